@@ -1,0 +1,166 @@
+"""The oracle's two layers pin each other on the TPC-H-shaped workloads.
+
+Layer 1 (interpreter running the Voodoo programs of oracle/programs.py) vs
+layer 2 (brute-force C loops) vs pandas / numpy (library) on generated
+tables.  Exact integer equality everywhere.
+"""
+import datetime
+
+import numpy as np
+import pandas as pd
+import pytest
+
+import gen
+import oracle
+from oracle import programs
+
+
+def lineitem(sf, seed=gen.DEFAULT_SEED):
+    n = gen.lineitem_rows(sf)
+    return {k: gen.host(c, n, sf=sf, seed=seed) for k, c in gen.LINEITEM_COLS.items()}
+
+
+def bind(p, prefix, cols):
+    for k, v in cols.items():
+        p.set(f"{prefix}.{k}", v)
+
+
+def pandas_q1(li, ship_max=10471):
+    df = pd.DataFrame({k: li[k].astype(object) if li[k].dtype == np.int64 else li[k] for k in li})
+    df = df[li["l_shipdate"] <= ship_max].copy()
+    df["k"] = df["l_returnflag"].astype(int) * 2 + df["l_linestatus"].astype(int)
+    df["dp"] = df["l_extendedprice"] * (100 - df["l_discount"])
+    df["ch"] = df["dp"] * (100 + df["l_tax"])
+    g = df.groupby("k").agg(q=("l_quantity", "sum"), b=("l_extendedprice", "sum"), dp=("dp", "sum"),
+                            ch=("ch", "sum"), d=("l_discount", "sum"), c=("l_quantity", "size"))
+    return {int(k): [int(x) for x in row] for k, row in zip(g.index, g.to_numpy())}
+
+
+@pytest.mark.parametrize("sf", [0.0002, 0.002])
+def test_q1_interpreter_bruteforce_pandas(sf):
+    li = lineitem(sf)
+    bf = oracle.q1(li)
+    assert bf == pandas_q1(li)
+    p = oracle.Program()
+    bind(p, "lineitem", li)
+    p.run(programs.Q1.format(ship_max_p1=10472))
+    keys = [k for k in p.get("o_key") if k is not None]
+    got = {k: [p.get(o)[j] for o in programs.Q1_OUTPUTS] for j, k in enumerate(keys)}
+    assert got == bf
+    assert keys == sorted(keys)  # ascending key order (reading A16)
+
+
+def test_q1_sharded_merge_equals_whole():
+    """Pin P8: row-range shards (the Fig 3 ctrl one level up)
+    merged by addition equal the whole-table result."""
+    sf = 0.002
+    li = lineitem(sf)
+    n = len(li["l_shipdate"])
+    whole = oracle.q1(li)
+    for G in [2, 3, 8]:
+        acc = {}
+        for r in range(G):
+            a, b = r * n // G, (r + 1) * n // G
+            part = oracle.q1({k: v[a:b] for k, v in li.items()})
+            for k, vals in part.items():
+                acc[k] = [x + y for x, y in zip(acc.get(k, [0] * 6), vals)]
+        assert acc == whole
+
+
+@pytest.mark.parametrize("intent", [1, 4, 1024, 10**9])
+def test_q6_interpreter_bruteforce_numpy(intent):
+    li = lineitem(0.002)
+    rev, cnt = oracle.q6(li)
+    m = ((li["l_shipdate"] >= 8766) & (li["l_shipdate"] < 9131) & (li["l_discount"] >= 5)
+         & (li["l_discount"] <= 7) & (li["l_quantity"] < 2400))
+    assert cnt == int(m.sum())
+    assert rev == int(np.sum(li["l_extendedprice"][m].astype(object) * li["l_discount"][m].astype(object)))
+    p = oracle.Program()
+    bind(p, "lineitem", li)
+    p.run(programs.Q6.format(intent=intent, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
+    assert p.get("revenue")[0] == rev
+    assert p.get("count")[0] == cnt
+
+
+@pytest.mark.parametrize("intent", [1, 32, 4096, 10**9])
+def test_select_sum_interpreter_bruteforce(intent):
+    n = 20000
+    v = gen.host(gen.F32_UNIFORM, n)
+    t = float(np.float32(0.5))
+    pos, c, (sh, sl) = oracle.select_f32(v, t, "lt")
+    assert pos.tolist() == np.flatnonzero(v < np.float32(t)).tolist()
+    p = oracle.Program()
+    p.set("input.val", v)
+    p.run(programs.SELECT_SUM.format(intent=intent, t=repr(t)))
+    assert p.get("count")[0] == c
+    got = p.get_float_exact("totalSum")
+    assert got[0][0] + got[1][0] == pytest.approx(sh + sl, rel=1e-15)
+    assert np.isclose(sh, np.sum(v[v < np.float32(t)], dtype=np.float64), rtol=1e-12)
+    sel = [x for x in p.get("positions") if x is not None]
+    assert sel == pos.tolist()  # runs concatenate to the global list
+
+
+def _dims(sf, seed=gen.DEFAULT_SEED):
+    npart, nsupp = gen.part_rows(sf), gen.supplier_rows(sf)
+    part = {k: gen.host(c, npart, sf=sf, seed=seed) for k, c in gen.PART_COLS.items()}
+    supp = {k: gen.host(c, nsupp, sf=sf, seed=seed) for k, c in gen.SUPPLIER_COLS.items()}
+    return part, supp
+
+
+def test_year_of_day_is_datetime():
+    for d in [0, 8035, 8400, 9131, 10561, 11000, 365, 730, 1095, 1461]:
+        assert oracle.year_of_day(d) == (datetime.date(1970, 1, 1) + datetime.timedelta(days=d)).year
+
+
+def test_fkj_q9_interpreter_bruteforce_pandas():
+    sf = 0.002
+    li = lineitem(sf)
+    part, supp = _dims(sf)
+    bf = oracle.fkj(1, li, part, supp)
+    # pandas: merge on dense FK positions, group by nation*7 + year-1992
+    df = pd.DataFrame({"s": li["l_suppkey"] - 1, "ship": li["l_shipdate"],
+                       "rev": li["l_extendedprice"].astype(object) * (100 - li["l_discount"]).astype(object)})
+    df["nat"] = supp["s_nationkey"][df["s"].to_numpy()].astype(int)
+    df["yr"] = [(datetime.date(1970, 1, 1) + datetime.timedelta(days=int(d))).year for d in df["ship"]]
+    df["g"] = df["nat"] * 7 + df["yr"] - 1992
+    g = df.groupby("g").agg(r=("rev", "sum"), c=("rev", "size"))
+    assert bf == {int(k): (int(r), int(c)) for k, (r, c) in zip(g.index, g.to_numpy())}
+    # interpreter with a calendar dimension (positional date -> year lookup)
+    day0 = 8000
+    cal = np.array([(datetime.date(1970, 1, 1) + datetime.timedelta(days=day0 + i)).year for i in range(3000)])
+    p = oracle.Program()
+    bind(p, "lineitem", li)
+    p.set("supplier.s_nationkey", supp["s_nationkey"])
+    p.set("calendar.year", cal)
+    p.run(programs.FKJ_Q9.format(day0=day0))
+    keys = [k for k in p.get("o_key") if k is not None]
+    got = {k: (p.get("o_rev")[j], p.get("o_cnt")[j]) for j, k in enumerate(keys)}
+    assert got == bf
+
+
+def test_fkj_q19_bruteforce_pandas():
+    sf = 0.01
+    li = lineitem(sf)
+    part, supp = _dims(sf)
+    bf = oracle.fkj(0, li, part, supp)
+    p = li["l_partkey"] - 1
+    brand = part["p_brand"][p]
+    cont = part["p_container"][p]
+    size = part["p_size"][p]
+    C = {s: i for i, s in enumerate(gen.CONTAINER)}
+    B = {s: i for i, s in enumerate(gen.BRAND)}
+    M = {s: i for i, s in enumerate(gen.SHIPMODE)}
+    I_ = {s: i for i, s in enumerate(gen.SHIPINSTRUCT)}
+    mode_ok = np.isin(li["l_shipmode"], [M[m] for m in ["AIR", "AIR REG"] if m in M])
+    instr_ok = li["l_shipinstruct"] == I_["DELIVER IN PERSON"]
+    q = li["l_quantity"]
+    m = np.zeros(len(q), dtype=bool)
+    for b, conts, qlo, smax in [("Brand#12", ["SM CASE", "SM BOX", "SM PACK", "SM PKG"], 1, 5),
+                                ("Brand#23", ["MED BAG", "MED BOX", "MED PKG", "MED PACK"], 10, 10),
+                                ("Brand#34", ["LG CASE", "LG BOX", "LG PACK", "LG PKG"], 20, 15)]:
+        m |= ((brand == B[b]) & np.isin(cont, [C[c] for c in conts]) & (q >= qlo * 100) & (q <= (qlo + 10) * 100)
+              & (size >= 1) & (size <= smax) & mode_ok & instr_ok)
+    rev = int(np.sum(li["l_extendedprice"][m].astype(object) * (100 - li["l_discount"][m]).astype(object)))
+    exp = {0: (rev, int(m.sum()))} if m.sum() else {}
+    assert bf == exp
+    assert m.sum() > 0  # the workload selects something at this size
