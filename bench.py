@@ -1,0 +1,453 @@
+#!/usr/bin/env python
+"""Benchmark of the Voodoo hot path on B200 (BASELINE.json metric).
+
+Default: TPC-H Q1 at SF100 (600 M lineitem rows, 22.8 GB of columns),
+row-range partitioned across the N GPUs of one node (one process per GPU,
+launched by torch.distributed.run for N > 1).  A step is one pass of the
+fused Q1 fragment over the whole table: predicate (a2), virtual
+Partition/Scatter (a5), grouped folds (a6/a7), the hierarchical fold down to
+one partials vector per GPU (a8) and, for N > 1, the NCCL all-gather of
+those partials (the cross-GPU exchange step).  Inputs are generated in HBM
+before the timed region (excluded) and are far larger
+than the 126 MB L2, so no flush is needed between steps.
+
+Prints ONE JSON line on rank 0 (the driver contract), with `roofline`,
+`cpu_baseline` (the oracle on a bounded sample), `clocks`, `e2e` and
+`gpu_launches`.  `--impl reference` times the CPU oracle (the tier's
+reference arm) on the same config and metric instead.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "rows/s and achieved HBM GB/s (% of peak) for TPC-H Q1/Q6 at 1/2/4/8 B200"
+
+# Algorithmic bytes per row: every
+# column each query reads, once.
+BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "q19": 4 + 3 * 8 + 1 + 1,
+                 "q9": 4 + 4 + 2 * 8}
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=None)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
+    ap.add_argument("--workload", default="q1", choices=["q1", "q6", "select", "q19", "q9"])
+    ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
+    ap.add_argument("--sel-mode", default="branch", choices=["branch", "predicated"])
+    ap.add_argument("--selectivity", type=float, default=0.5, help="select workload: fraction selected")
+    ap.add_argument("--rows", type=int, default=None, help="select workload: rows (default 1e9)")
+    ap.add_argument("--generic", action="store_true", help="force the generic fragment")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--cpu-seconds", type=float, default=10.0)
+    ap.add_argument("--seed", type=int, default=0x5EEDC0DE)
+    return ap.parse_args()
+
+
+def default_sf(w):
+    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0}[w]
+
+
+# ---------------------------------------------------------------------------
+# measured peaks (driver-written)
+# ---------------------------------------------------------------------------
+def hbm_peak():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            return float(json.load(f)["hbm_gbs"]), "measured"
+    except Exception:
+        return 6650.0, "fallback"
+
+
+def ncu_traffic(workload):
+    """dram bytes per launch of the dominant kernel from the committed
+    `ncu --set full` summary (profiles/ncu_summary.json), else None."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_summary.json")) as f:
+            d = json.load(f)
+        return d.get(workload, {}).get("dram_bytes_per_launch")
+    except Exception:
+        return None
+
+
+# ---------------------------------------------------------------------------
+# clocks sampled during the timed region
+# ---------------------------------------------------------------------------
+class ClockSampler:
+    FIELDS = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+              "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, dev):
+        self.dev = dev
+        self.proc = None
+        self.lines = []
+        self.t = None
+
+    def start(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", f"--query-gpu={self.FIELDS}", "--format=csv,noheader,nounits",
+                                          "-lms", "100", "-i", str(self.dev)], stdout=subprocess.PIPE,
+                                         stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def stop(self):
+        if self.proc is None:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["nvidia-smi unavailable"]}
+        self.proc.terminate()
+        try:
+            self.proc.wait(timeout=5)
+        except Exception:
+            self.proc.kill()
+        if self.t:
+            self.t.join(timeout=2)
+        sm, mx, reasons = [], [], set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for ln in self.lines:
+            p = [x.strip() for x in ln.split(",")]
+            if len(p) < 9:
+                continue
+            try:
+                sm.append(float(p[1]))
+                mx.append(float(p[2]))
+            except ValueError:
+                continue
+            for nm, v in zip(names, p[5:9]):
+                if v.lower() == "active":
+                    reasons.add(nm)
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": sorted(reasons), "samples": len(sm)}
+
+
+# ---------------------------------------------------------------------------
+# CPU oracle baseline (bounded sample)
+# ---------------------------------------------------------------------------
+def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5):
+    """Time the oracle as it stands (the literal Voodoo interpreter, one
+    thread) on chunks of the same workload until ~budget_s of CPU work."""
+    import numpy as np
+
+    import gen
+    import oracle
+    from oracle import programs
+
+    chunk = 1 << 19
+    rows_done, t_total = 0, 0.0
+    row0 = 0
+    n_total = gen.lineitem_rows(sf) if workload != "select" else 10**9
+    while t_total < budget_s and row0 < n_total:
+        m = min(chunk, n_total - row0)
+        if workload == "select":
+            v = gen.host(gen.F32_UNIFORM, m, row0, seed=seed)
+            t0 = time.perf_counter()
+            p = oracle.Program()
+            p.set("input.val", v)
+            p.run(programs.SELECT_SUM.format(intent=m, t=float(np.float32(sel_t)).hex()))
+            t_total += time.perf_counter() - t0
+        else:
+            li = {k: gen.host(c, m, row0, sf=sf, seed=seed) for k, c in gen.LINEITEM_COLS.items()}
+            t0 = time.perf_counter()
+            p = oracle.Program()
+            for k, v in li.items():
+                p.set("lineitem." + k, v)
+            if workload == "q1":
+                p.run(programs.Q1.format(ship_max_p1=10472))
+            elif workload == "q6":
+                p.run(programs.Q6.format(intent=1 << 30, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
+            else:
+                oracle.q1(li)  # FKJ: brute-force layer (interpreter needs a calendar dim)
+            t_total += time.perf_counter() - t0
+        rows_done += m
+        row0 += m
+    return {"value": rows_done / t_total, "unit": "rows/s", "cores": 1, "kind": "oracle",
+            "sample": f"{rows_done} rows of the {workload} workload (rows 0..{rows_done - 1}, chunks of {chunk}), "
+                      f"literal Voodoo interpreter (oracle/voodoo_oracle.cpp), {t_total:.1f} s single-threaded",
+            "seconds": t_total}
+
+
+# ---------------------------------------------------------------------------
+# the GPU arm
+# ---------------------------------------------------------------------------
+def main():
+    args = parse()
+    rank = int(os.environ.get("RANK", "0"))
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    sf = args.sf if args.sf is not None else default_sf(args.workload)
+
+    if args.impl == "reference":
+        return reference_arm(args, rank, world, sf)
+
+    import torch
+    import torch.distributed as dist
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+    stream = torch.cuda.current_stream()
+
+    w = args.workload
+    if w == "select":
+        n_total = args.rows or 10**9
+    else:
+        n_total = gen.lineitem_rows(sf)
+    a, b = rank * n_total // world, (rank + 1) * n_total // world
+    n = b - a
+    sel_mode = vd.VD_SEL_PREDICATED if args.sel_mode == "predicated" else vd.VD_SEL_BRANCH
+
+    # ---- a1: columns generated in HBM (row range [a, b)), min/max via vd folds
+    def make(col, length, row0, sfv=sf, **kw):
+        t = torch.empty(length, dtype=getattr(torch, _dt(col)), device=dev)
+        gen.device(col, t.data_ptr(), length, row0, sf=sfv, seed=args.seed, stream=stream.cuda_stream, **kw)
+        return t
+
+    def meta(t):
+        c = vd.column(t)
+        if c.dtype in (vd.VD_F32, vd.VD_F64) or t.numel() == 0:
+            return c
+        lo = torch.empty(1, dtype=t.dtype, device=dev)
+        hi = torch.empty(1, dtype=t.dtype, device=dev)
+        vd.fold_min(c, None, out=lo)
+        vd.fold_max(c, None, out=hi)
+        return vd.column(t, minmax=(int(lo.item()), int(hi.item())))
+
+    dims, dim_views, cols = [], [], []
+    if w == "q1":
+        names, plan = plans.Q1_COLS, plans.q1(sel_mode, force_generic=args.generic)
+    elif w == "q6":
+        names, plan = plans.Q6_COLS, plans.q6(sel_mode, force_generic=args.generic)
+    elif w == "q19":
+        names = plans.Q19_COLS
+        plan = plans.q19({"brand": {s: i for i, s in enumerate(gen.BRAND)},
+                          "container": {s: i for i, s in enumerate(gen.CONTAINER)},
+                          "shipmode": {s: i for i, s in enumerate(gen.SHIPMODE)},
+                          "shipinstruct": {s: i for i, s in enumerate(gen.SHIPINSTRUCT)}}, sel_mode,
+                         force_generic=args.generic)
+        for d in plans.Q19_DIMS:
+            dims.append(make(gen.PART_COLS[d], gen.part_rows(sf), 0))
+    elif w == "q9":
+        names, plan = plans.Q9_COLS, plans.q9(sel_mode, force_generic=args.generic)
+        for d in plans.Q9_DIMS:
+            dims.append(make(gen.SUPPLIER_COLS[d], gen.supplier_rows(sf), 0))
+    else:
+        names = ["v"]
+        plan = plans.selsum(float(__import__("numpy").float32(args.selectivity)), sel_mode,
+                            force_generic=args.generic)
+    for nm in names:
+        col = gen.F32_UNIFORM if nm == "v" else gen.LINEITEM_COLS[nm]
+        cols.append(make(col, n, a))
+    torch.cuda.synchronize()
+    views = [meta(t) for t in cols]
+    dim_views = [meta(t) for t in dims]
+    torch.cuda.synchronize()
+
+    pbytes = vd.partials_bytes(plan)
+    out = torch.empty(pbytes, dtype=torch.uint8, device=dev)
+    ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
+    gathered = torch.empty(pbytes * world, dtype=torch.uint8, device=dev) if world > 1 else None
+
+    def step():
+        vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
+        if world > 1:
+            dist.all_gather_into_tensor(gathered, out)
+
+    steps = args.steps if args.steps is not None else (300 if w in ("q1", "q19", "q9") else 1000)
+    for _ in range(max(args.warmup, 0)):
+        step()
+    launches_per_step = vd.last_launch_count()
+    torch.cuda.synchronize()
+
+    # ---- timed region --------------------------------------------------------
+    clocks = ClockSampler(local)
+    clocks.start()
+    time.sleep(0.3)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(steps)]
+    t_start = torch.cuda.Event(enable_timing=True)
+    t_end = torch.cuda.Event(enable_timing=True)
+    wall0 = time.perf_counter()
+    t_start.record(stream)
+    for i in range(steps):
+        ev[i][0].record(stream)
+        vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
+        ev[i][1].record(stream)
+        if world > 1:
+            dist.all_gather_into_tensor(gathered, out)
+    t_end.record(stream)
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    wall = time.perf_counter() - wall0
+    clk = clocks.stop()
+    elapsed_ms = t_start.elapsed_time(t_end)
+    kernel_ms = sum(s.elapsed_time(e) for s, e in ev) / steps
+    if world > 1:
+        tt = torch.tensor([elapsed_ms, kernel_ms], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        elapsed_ms, kernel_ms = float(tt[0]), float(tt[1])
+    ms_per_step = elapsed_ms / steps
+
+    # result check (merge of the per-rank partials, host side)
+    if world > 1:
+        parts = [gathered[r * pbytes:(r + 1) * pbytes].cpu().numpy().tobytes() for r in range(world)]
+        merged = vd.merge_partials(plan, views, dim_views, parts)
+    else:
+        merged = out.cpu().numpy().tobytes()
+    fl = [w == "select"] + [False] * 8
+    result = vd.decode_partials(merged, plan, float_aggs=fl)
+
+    # ---- e2e: host buffers in, result out, through the public API -------------
+    e2e = None
+    if not args.no_e2e:
+        e2e = e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, dist, pbytes)
+
+    peak, peak_kind = hbm_peak()
+    bpr = BYTES_PER_ROW[w]
+    achieved = n * bpr / (kernel_ms * 1e-3) / 1e9  # per GPU, dominant-kernel duration
+    rows_per_s = n_total / (ms_per_step * 1e-3)
+    line = {
+        "metric": METRIC,
+        "value": rows_per_s,
+        "unit": "rows/s",
+        "n_gpus": world,
+        "steps": steps,
+        "warmup": args.warmup,
+        "ms_per_step": ms_per_step,
+        "higher_is_better": True,
+        "scaling": "strong",
+        "vs_baseline": None,
+        "dtype": "f32/f64" if w == "select" else "int64",
+        "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
+        "config": {
+            "workload": {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
+                         "q9": f"fkj_q9_sf{sf:g}", "select": f"select_f32_{n_total}_s{args.selectivity:g}"}[w],
+            "rows": n_total, "rows_per_gpu": n, "sf": sf, "sel_mode": args.sel_mode,
+            "fragment": "generic" if args.generic else "specialised",
+            "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
+            "l2": f"inputs {n * bpr / 1e9:.1f} GB per GPU > 126 MB L2: no flush needed",
+            "seed": args.seed,
+        },
+        "hbm_gbs": achieved,
+        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                     "frac": achieved / peak, "peak_kind": peak_kind,
+                     "traffic": ncu_traffic(w), "bytes_per_row": bpr,
+                     "kernel": "k_pipe_q1+k_q1_remap" if w == "q1" and not args.generic else "vd_run_pipeline",
+                     "kernel_ms": kernel_ms},
+        "clocks": clk,
+        "e2e": e2e,
+        "gpu_launches": launches_per_step * steps,
+        "result": {str(k): [str(x) for x in v] for k, v in list(result.items())[:8]},
+        "wall_s": wall,
+    }
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        line["cpu_baseline"] = cpu_baseline(w, sf if w != "select" else 0, args.seed, args.cpu_seconds,
+                                            args.selectivity)
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.barrier()
+        dist.destroy_process_group()
+
+
+def _dt(col):
+    import gen
+    import numpy as np
+    return {np.uint8: "uint8", np.int32: "int32", np.int64: "int64", np.float32: "float32",
+            np.float64: "float64"}[gen.dtype_of(col)]
+
+
+def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, dist, pbytes):
+    """Through the public API from pinned host buffers: vd_load_column (H2D)
+    of every input column, vd_run_pipeline, D2H of the partials."""
+    try:
+        host = [torch.empty(c.numel(), dtype=c.dtype, pin_memory=True) for c in cols]
+        pinned = True
+    except Exception:
+        host = [torch.empty(c.numel(), dtype=c.dtype) for c in cols]
+        pinned = False
+    for h, c in zip(host, cols):
+        h.copy_(c)
+    dst = [torch.empty_like(c) for c in cols]
+    out = torch.empty(pbytes, dtype=torch.uint8, device=dev)
+    res = torch.empty(pbytes, dtype=torch.uint8, pin_memory=pinned)
+    ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
+    reps = 3
+    torch.cuda.synchronize()
+    if world > 1:
+        dist.barrier()
+    t0 = time.perf_counter()
+    for _ in range(reps):
+        vcols = []
+        for h, d, v in zip(host, dst, views):
+            c = vd.load_column(h, d, compute_minmax=False, stream=stream)
+            c.min, c.max, c.has_minmax = v.min, v.max, v.has_minmax  # catalog metadata
+            vcols.append(c)
+        vd.run_pipeline(plan, vcols, n, dim_views, out=out, ws=ws, stream=stream)
+        res.copy_(out, non_blocking=True)
+        torch.cuda.synchronize()
+    dt = (time.perf_counter() - t0) / reps
+    if world > 1:
+        t = torch.tensor([dt], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        dt = float(t[0])
+    h2d = sum(c.numel() * c.element_size() for c in cols)
+    del host, dst
+    return {"value": (n * world) / dt, "unit": "rows/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": pbytes,
+            "pinned": pinned, "reps": reps, "s_per_step": dt}
+
+
+def reference_arm(args, rank, world, sf):
+    """The tier's reference arm: the CPU oracle on the same config/metric."""
+    if rank != 0:
+        return
+    w = args.workload
+    steps = args.steps if args.steps is not None else 3
+    budget = max(1.0, min(args.cpu_seconds, 60.0) / max(steps, 1))
+    vals = []
+    cb = None
+    if args.warmup > 0:
+        cpu_baseline(w, sf if w != "select" else 0, args.seed, 0.5, args.selectivity)
+    t0 = time.perf_counter()
+    for _ in range(steps):
+        cb = cpu_baseline(w, sf if w != "select" else 0, args.seed, budget, args.selectivity)
+        vals.append(cb["value"])
+    wall = time.perf_counter() - t0
+    v = statistics.median(vals)
+    line = {"metric": METRIC, "value": v, "unit": "rows/s", "impl": "reference", "n_gpus": world, "steps": steps,
+            "warmup": args.warmup, "ms_per_step": wall / steps * 1e3, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "int64", "data": "synthetic",
+            "config": {"workload": {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
+                                    "q9": f"fkj_q9_sf{sf:g}", "select": "select_f32"}[w], "sf": sf},
+            "cpu_baseline": {"value": v, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": cb["sample"]},
+            "e2e": {"value": v, "unit": "rows/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+if __name__ == "__main__":
+    main()

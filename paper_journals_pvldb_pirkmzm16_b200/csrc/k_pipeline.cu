@@ -1,0 +1,1127 @@
+// k_pipeline.cu -- fused operator chains, vd_run_pipeline (§8(a) a7-a9).
+//
+// A Voodoo fragment (§3.1) is one fully inlined kernel: scan ->
+// predicate -> (FK gather) -> group key -> folds, with materialisation only
+// at the seams.  Here the fragments are compiled ahead of time for sm_100a:
+//
+//   k_pipe_q1      grouped multi-aggregate over <= 8 groups (the Q1 plan of
+//                  Fig 10/11): the Partition -> Scatter -> FoldSum/FoldCount
+//                  chain stays virtual (§3.1.3) -- each row's
+//                  values go straight into its group's register accumulators
+//                  (the "scatter position" is the work-item-local key), and
+//                  the FoldSelect compaction happens on the host merge.
+//   k_pipe_scalar  filtered scalar fold of a product of columns (the Q6 plan
+//                  of Fig 8, and the selective aggregation of
+//                  Fig 15), branching (late loads) or
+//                  predicated (every row loaded, contribution x predicate).
+//   k_pipe_generic any vd_pipeline: per-row interpretation of the descriptor
+//                  (gathers, key parts, products), per-warp shared-memory
+//                  accumulators updated by one leader lane per distinct key.
+//
+// Hierarchical fold (Fig 3): thread -> warp -> CTA partials in
+// the workspace -> the last CTA to finish folds them in CTA order (Fragment 2
+// / global barrier) and writes the vd_partials buffer.
+#include <float.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstring>
+
+#include "vd_common.cuh"
+#include "vd_internal.h"
+#include "vd_pred.cuh"
+
+namespace vd {
+
+// ============================================================================
+// Output slots
+// ============================================================================
+// partials: [ngroups][naggs+1] x 16 bytes (include/vd.h vd_partials).
+struct Slot16 {
+    unsigned long long lo, hi;
+};
+
+__device__ __forceinline__ void put_i128(Slot16* s, i128 v) {
+    s->lo = (unsigned long long)(u128)v;
+    s->hi = (unsigned long long)((u128)v >> 64);
+}
+__device__ __forceinline__ i128 get_i128(const Slot16& s) { return (i128)(((u128)s.hi << 64) | s.lo); }
+__device__ __forceinline__ void put_f64(Slot16* s, double v) {
+    s->lo = (unsigned long long)__double_as_longlong(v);
+    s->hi = 0;
+}
+__device__ __forceinline__ double get_f64(const Slot16& s) { return __longlong_as_double((long long)s.lo); }
+
+// ============================================================================
+// Generic fragment
+// ============================================================================
+struct GenAgg {
+    int32_t kind, nf, isf;
+    int32_t col[VD_MAX_FACTORS];
+    int64_t a[VD_MAX_FACTORS], b[VD_MAX_FACTORS];
+};
+
+struct GenPlan {
+    DevPred pred;
+    DevCols cols;  // base columns
+    // gathers
+    int32_t ngathers;
+    int32_t g_fk[VD_MAX_GATHERS];
+    int64_t g_bias[VD_MAX_GATHERS];
+    const void* g_p[VD_MAX_GATHERS];
+    int64_t g_len[VD_MAX_GATHERS];
+    int32_t g_dt[VD_MAX_GATHERS];
+    // key
+    int32_t nkey;
+    int32_t k_col[VD_MAX_KEYPARTS], k_fn[VD_MAX_KEYPARTS];
+    int64_t k_sub[VD_MAX_KEYPARTS], k_mult[VD_MAX_KEYPARTS];
+    int64_t ngroups;
+    int32_t naggs;
+    GenAgg agg[VD_MAX_AGGS];
+};
+
+__device__ __forceinline__ Val gen_fetch(const GenPlan& P, int c, int64_t row) {
+    if (c < P.cols.ncols) return fetch_typed(P.cols.p[c], P.cols.dt[c], row);
+    int g = c - P.cols.ncols;
+    Val fk = fetch_typed(P.cols.p[P.g_fk[g]], P.cols.dt[P.g_fk[g]], row);
+    Val out;
+    out.eps = true;
+    out.isf = false;
+    out.i = 0;
+    out.f = 0;
+    if (fk.eps) return out;
+    int64_t p = fk.i - P.g_bias[g];
+    if (p < 0 || p >= P.g_len[g]) return out;
+    return fetch_typed(P.g_p[g], P.g_dt[g], p);
+}
+
+__device__ __forceinline__ bool gen_pred(const GenPlan& P, int64_t row) {
+    if (P.pred.nconj == 0) return true;
+    for (int c = 0; c < P.pred.nconj; ++c) {
+        bool ok = true;
+        for (int k = 0; k < P.pred.nterms[c] && ok; ++k) {
+            const DevTerm& t = P.pred.t[c][k];
+            ok = term_true(t, gen_fetch(P, t.col, row));
+        }
+        if (ok) return true;
+    }
+    return false;
+}
+
+constexpr int GEN_THREADS = 256;
+constexpr int GEN_WARPS = GEN_THREADS / 32;
+
+// Accumulator slot layout per (group, agg): 16 bytes (i128 or f64/i64 min-max);
+// slot [g][naggs] = row count.
+template <bool SMEM>
+__global__ void __launch_bounds__(GEN_THREADS) k_pipe_generic(const __grid_constant__ GenPlan P, int64_t n,
+                                                              Slot16* __restrict__ block_parts, int nslots,
+                                                              Slot16* __restrict__ gacc,
+                                                              unsigned long long* __restrict__ gmask,
+                                                              unsigned int* __restrict__ done, Slot16* __restrict__ out,
+                                                              unsigned long long* __restrict__ domain_err) {
+    extern __shared__ Slot16 s_mem[];
+    // [GEN_WARPS][32][naggs] staging, then (SMEM) [GEN_WARPS][nslots] accumulators
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int NA = P.naggs;
+    Slot16* stage = s_mem + (size_t)warp * 32 * (NA + 1);
+    Slot16* acc = s_mem + (size_t)GEN_WARPS * 32 * (NA + 1) + (size_t)warp * nslots;
+    if (SMEM) {
+        for (int k = lane; k < nslots; k += 32) {
+            int a = k % (NA + 1);
+            Slot16 z{0, 0};
+            if (a < NA && (P.agg[a].kind == VD_AGG_MIN || P.agg[a].kind == VD_AGG_MAX)) {
+                bool mn = P.agg[a].kind == VD_AGG_MIN;
+                if (P.agg[a].isf) put_f64(&z, mn ? DBL_MAX : -DBL_MAX);
+                else put_i128(&z, mn ? (i128)INT64_MAX : (i128)INT64_MIN);
+            }
+            acc[k] = z;
+        }
+    }
+    __syncwarp();
+    const int64_t stride = (int64_t)gridDim.x * GEN_THREADS;
+    for (int64_t base = (int64_t)blockIdx.x * GEN_THREADS + warp * 32; base < n; base += stride) {
+        const int64_t row = base + lane;
+        bool ok = row < n && gen_pred(P, row);
+        int64_t key = 0;
+        if (ok) {
+            for (int k = 0; k < P.nkey && ok; ++k) {
+                Val v = gen_fetch(P, P.k_col[k], row);
+                if (v.eps) { ok = false; break; }
+                int64_t x = v.isf ? (int64_t)v.f : v.i;
+                if (P.k_fn[k] == 1) x = year_of_day((int32_t)x);
+                key += (x - P.k_sub[k]) * P.k_mult[k];
+            }
+            if (ok && (key < 0 || key >= P.ngroups)) {
+                ok = false;
+                atomicAdd(domain_err, 1ull);
+            }
+        }
+        if (ok) {
+            for (int a = 0; a < NA; ++a) {
+                const GenAgg& A = P.agg[a];
+                Slot16 v{0, 0};
+                if (A.kind == VD_AGG_COUNT) {
+                    put_i128(&v, 1);
+                } else if (A.isf) {
+                    double pr = 1.0;
+                    bool e = false;
+                    for (int f = 0; f < A.nf; ++f) {
+                        double x = 0;
+                        if (A.col[f] >= 0) {
+                            Val c = gen_fetch(P, A.col[f], row);
+                            e |= c.eps;
+                            x = c.isf ? c.f : (double)c.i;
+                        }
+                        pr *= (double)A.a[f] + (double)A.b[f] * x;
+                    }
+                    if (e) pr = nan("");
+                    put_f64(&v, pr);
+                } else {
+                    i128 pr = 1;
+                    bool e = false;
+                    for (int f = 0; f < A.nf; ++f) {
+                        i128 x = 0;
+                        if (A.col[f] >= 0) {
+                            Val c = gen_fetch(P, A.col[f], row);
+                            e |= c.eps;
+                            x = c.i;
+                        }
+                        pr *= (i128)A.a[f] + (i128)A.b[f] * x;
+                    }
+                    put_i128(&v, pr);
+                    if (e) v.hi = 0x8000000000000000ull;  // epsilon marker (skipped)
+                }
+                stage[lane * (NA + 1) + a] = v;
+            }
+        }
+        __syncwarp();
+        unsigned m = __match_any_sync(VD_FULL, ok ? key : -1ll);
+        bool leader = ok && (__ffs(m) - 1 == lane);
+        if (leader) {
+            for (int a = 0; a <= NA; ++a) {
+                const bool cnt = (a == NA);
+                const int kind = cnt ? VD_AGG_COUNT : P.agg[a].kind;
+                const bool isf = cnt ? false : P.agg[a].isf;
+                Slot16 r;
+                if (SMEM) r = acc[key * (NA + 1) + a];
+                i128 si = 0, mi = 0;
+                double sf = 0, mf = 0;
+                bool have = false;
+                for (unsigned mm = m; mm; mm &= mm - 1) {
+                    int l = __ffs(mm) - 1;
+                    if (cnt) { si += 1; continue; }
+                    Slot16 x = stage[l * (NA + 1) + a];
+                    if (!isf && x.hi == 0x8000000000000000ull && kind != VD_AGG_COUNT) continue;
+                    if (isf && kind != VD_AGG_COUNT) {
+                        double d = get_f64(x);
+                        if (d != d) continue;
+                        if (kind == VD_AGG_SUM) sf += d;
+                        else if (!have || (kind == VD_AGG_MIN ? d < mf : d > mf)) mf = d;
+                    } else {
+                        i128 y = get_i128(x);
+                        if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) si += y;
+                        else if (!have || (kind == VD_AGG_MIN ? y < mi : y > mi)) mi = y;
+                    }
+                    have = true;
+                }
+                if (SMEM) {
+                    if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) {
+                        if (isf) put_f64(&r, get_f64(r) + sf);
+                        else put_i128(&r, get_i128(r) + si);
+                    } else if (have) {
+                        if (isf) { double c = get_f64(r); put_f64(&r, kind == VD_AGG_MIN ? fmin(c, mf) : fmax(c, mf)); }
+                        else { i128 c = get_i128(r); put_i128(&r, kind == VD_AGG_MIN ? (mi < c ? mi : c) : (mi > c ? mi : c)); }
+                    }
+                    acc[key * (NA + 1) + a] = r;
+                } else {
+                    unsigned long long* g = (unsigned long long*)(gacc + key * (NA + 1) + a);
+                    if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) {
+                        if (isf) atomicAdd((double*)g, sf);
+                        else atomic_add_i128(g, si);
+                    } else if (have) {
+                        if (isf) {
+                            // order-preserving integer image of a double
+                            long long bits = __double_as_longlong(mf);
+                            long long key2 = bits >= 0 ? bits : bits ^ 0x7FFFFFFFFFFFFFFFll;
+                            if (kind == VD_AGG_MIN) atomicMin((long long*)g, key2); else atomicMax((long long*)g, key2);
+                        } else {
+                            if (kind == VD_AGG_MIN) atomicMin((long long*)g, (long long)mi);
+                            else atomicMax((long long*)g, (long long)mi);
+                        }
+                        atomicOr(gmask + key * (NA + 1) + a, 1ull);
+                    }
+                }
+            }
+        }
+        __syncwarp();
+    }
+    if (!SMEM) {
+        // the last CTA converts min/max images and copies to out
+        __syncthreads();
+        __shared__ bool s_last;
+        if (threadIdx.x == 0) {
+            __threadfence();
+            s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+        }
+        __syncthreads();
+        if (!s_last) return;
+        __threadfence();
+        for (int k = threadIdx.x; k < P.ngroups * (NA + 1); k += GEN_THREADS) {
+            int a = k % (NA + 1);
+            Slot16 v;
+            v.lo = __ldcg(&gacc[k].lo);
+            v.hi = __ldcg(&gacc[k].hi);
+            if (a < NA && (P.agg[a].kind == VD_AGG_MIN || P.agg[a].kind == VD_AGG_MAX)) {
+                if (P.agg[a].isf) {
+                    long long key2 = (long long)v.lo;
+                    long long bits = key2 >= 0 ? key2 : key2 ^ 0x7FFFFFFFFFFFFFFFll;
+                    put_f64(&v, __longlong_as_double(bits));
+                } else {
+                    put_i128(&v, (i128)(long long)v.lo);
+                }
+            }
+            out[k] = v;
+        }
+        return;
+    }
+    // fold the warps' accumulators into this CTA's partial, then the grid's
+    __syncthreads();
+    Slot16* wacc = s_mem + (size_t)GEN_WARPS * 32 * (NA + 1);
+    for (int k = threadIdx.x; k < nslots; k += GEN_THREADS) {
+        int a = k % (NA + 1);
+        const bool cnt = (a == NA);
+        const int kind = cnt ? VD_AGG_COUNT : P.agg[a].kind;
+        const bool isf = cnt ? false : P.agg[a].isf;
+        Slot16 r = wacc[k];
+        for (int w = 1; w < GEN_WARPS; ++w) {
+            Slot16 x = wacc[(size_t)w * nslots + k];
+            if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) {
+                if (isf) put_f64(&r, get_f64(r) + get_f64(x)); else put_i128(&r, get_i128(r) + get_i128(x));
+            } else if (isf) {
+                put_f64(&r, kind == VD_AGG_MIN ? fmin(get_f64(r), get_f64(x)) : fmax(get_f64(r), get_f64(x)));
+            } else {
+                i128 p = get_i128(r), q = get_i128(x);
+                put_i128(&r, kind == VD_AGG_MIN ? (q < p ? q : p) : (q > p ? q : p));
+            }
+        }
+        block_parts[(size_t)blockIdx.x * nslots + k] = r;
+    }
+    __shared__ bool s_last2;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last2 = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last2) return;
+    __threadfence();
+    for (int k = threadIdx.x; k < nslots; k += GEN_THREADS) {
+        int a = k % (NA + 1);
+        const bool cnt = (a == NA);
+        const int kind = cnt ? VD_AGG_COUNT : P.agg[a].kind;
+        const bool isf = cnt ? false : P.agg[a].isf;
+        Slot16 r;
+        r.lo = __ldcg(&block_parts[k].lo);
+        r.hi = __ldcg(&block_parts[k].hi);
+        for (unsigned b = 1; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&block_parts[(size_t)b * nslots + k].lo);
+            x.hi = __ldcg(&block_parts[(size_t)b * nslots + k].hi);
+            if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) {
+                if (isf) put_f64(&r, get_f64(r) + get_f64(x)); else put_i128(&r, get_i128(r) + get_i128(x));
+            } else if (isf) {
+                put_f64(&r, kind == VD_AGG_MIN ? fmin(get_f64(r), get_f64(x)) : fmax(get_f64(r), get_f64(x)));
+            } else {
+                i128 p = get_i128(r), q = get_i128(x);
+                put_i128(&r, kind == VD_AGG_MIN ? (q < p ? q : p) : (q > p ? q : p));
+            }
+        }
+        out[k] = r;
+    }
+}
+
+// ============================================================================
+// Q1-shaped fragment: <= G groups from two u8 key columns, predicate an
+// interval on one i32 column, aggregates from four i64 columns V0..V3:
+//   S0 = SUM(V0)                          (sum_qty)
+//   S1 = SUM(V1)                          (sum_base_price)
+//   S2 = SUM(V1*(a1 + b1*V2))             (sum_disc_price)
+//   S3 = SUM(V1*(a1 + b1*V2)*(a2 + b2*V3))(sum_charge)
+//   S4 = SUM(V2)                          (sum_disc)
+//   S5 = COUNT                            (count_order)
+// ============================================================================
+struct Q1Args {
+    const int32_t* d;  // predicate column
+    int32_t dlo, dhi;  // lo <= d <= hi
+    const uint8_t* k1;
+    const uint8_t* k2;
+    int32_t m1, m2, koff;  // key = k1*m1 + k2*m2 + koff
+    const int64_t* v[4];
+    int64_t a1, b1, a2, b2;
+    int64_t nquads;  // n / 4 (full quads); the tail is handled by the last CTA
+    int64_t n;
+};
+
+constexpr int Q1_THREADS = 256;
+
+// packed (disc, count) accumulator: disc in bits 0..39, count in bits 40..63
+constexpr int Q1_CSHIFT = 40;
+
+template <int G, bool NARROW>
+struct Q1Acc {
+    int64_t s0[G], s1[G], s2[G], s3[G], dc[G];
+};
+
+template <int G, bool NARROW>
+__device__ __forceinline__ void q1_row(Q1Acc<G, NARROW>& A, const Q1Args& a, bool pass, int key, int64_t v0,
+                                       int64_t v1, int64_t v2, int64_t v3) {
+    int64_t dp, ch;
+    if (NARROW) {
+        // metadata proves |V1|, |a1+b1*V2|, |dp|, |a2+b2*V3| < 2^31 and the
+        // constants fit in 32 bits: the factors are exact in wrapping 32-bit
+        // arithmetic and each product is one 32x32->64 IMAD.WIDE
+        int32_t f1 = (int32_t)a.a1 + (int32_t)a.b1 * (int32_t)v2;
+        dp = (int64_t)(int32_t)v1 * (int64_t)f1;
+        int32_t f2 = (int32_t)a.a2 + (int32_t)a.b2 * (int32_t)v3;
+        ch = (int64_t)(int32_t)dp * (int64_t)f2;
+    } else {
+        dp = v1 * (a.a1 + a.b1 * v2);
+        ch = dp * (a.a2 + a.b2 * v3);
+    }
+    const int64_t dc = v2 + (1ll << Q1_CSHIFT);
+#pragma unroll
+    for (int g = 0; g < G; ++g) {
+        if (pass && key == g) {
+            A.s0[g] += v0;
+            A.s1[g] += v1;
+            A.s2[g] += dp;
+            A.s3[g] += ch;
+            A.dc[g] += dc;
+        }
+    }
+}
+
+template <int G, bool NARROW>
+__global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant__ Q1Args a, Slot16* __restrict__ parts,
+                                                           unsigned int* __restrict__ done, Slot16* __restrict__ out) {
+    Q1Acc<G, NARROW> A;
+#pragma unroll
+    for (int g = 0; g < G; ++g) { A.s0[g] = A.s1[g] = A.s2[g] = A.s3[g] = A.dc[g] = 0; }
+
+    const int64_t nthreads = (int64_t)gridDim.x * Q1_THREADS;
+    const int64_t tid = (int64_t)blockIdx.x * Q1_THREADS + threadIdx.x;
+    // two quads in flight per thread per iteration (q and q + nthreads)
+    int64_t q = tid;
+    for (; q + nthreads < a.nquads; q += 2 * nthreads) {
+        int4 d[2];
+        uint32_t k1[2], k2[2];
+        longlong2 x[2][4][2];
+#pragma unroll
+        for (int u = 0; u < 2; ++u) {
+            const int64_t qq = q + u * nthreads;
+            d[u] = __ldg(reinterpret_cast<const int4*>(a.d) + qq);
+            k1[u] = __ldg(reinterpret_cast<const unsigned int*>(a.k1) + qq);
+            k2[u] = __ldg(reinterpret_cast<const unsigned int*>(a.k2) + qq);
+#pragma unroll
+            for (int c = 0; c < 4; ++c) {
+                x[u][c][0] = __ldg(reinterpret_cast<const longlong2*>(a.v[c]) + 2 * qq);
+                x[u][c][1] = __ldg(reinterpret_cast<const longlong2*>(a.v[c]) + 2 * qq + 1);
+            }
+        }
+#pragma unroll
+        for (int u = 0; u < 2; ++u) {
+            const int dd[4] = {d[u].x, d[u].y, d[u].z, d[u].w};
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                bool pass = dd[j] >= a.dlo && dd[j] <= a.dhi;
+                int key = (int)((k1[u] >> (8 * j)) & 0xFF) * a.m1 + (int)((k2[u] >> (8 * j)) & 0xFF) * a.m2 + a.koff;
+                int64_t v0 = (j & 1) ? x[u][0][j >> 1].y : x[u][0][j >> 1].x;
+                int64_t v1 = (j & 1) ? x[u][1][j >> 1].y : x[u][1][j >> 1].x;
+                int64_t v2 = (j & 1) ? x[u][2][j >> 1].y : x[u][2][j >> 1].x;
+                int64_t v3 = (j & 1) ? x[u][3][j >> 1].y : x[u][3][j >> 1].x;
+                q1_row<G, NARROW>(A, a, pass, key, v0, v1, v2, v3);
+            }
+        }
+    }
+    for (; q < a.nquads; q += nthreads) {
+        int4 d = __ldg(reinterpret_cast<const int4*>(a.d) + q);
+        uint32_t k1 = __ldg(reinterpret_cast<const unsigned int*>(a.k1) + q);
+        uint32_t k2 = __ldg(reinterpret_cast<const unsigned int*>(a.k2) + q);
+        longlong2 x[4][2];
+#pragma unroll
+        for (int c = 0; c < 4; ++c) {
+            x[c][0] = __ldg(reinterpret_cast<const longlong2*>(a.v[c]) + 2 * q);
+            x[c][1] = __ldg(reinterpret_cast<const longlong2*>(a.v[c]) + 2 * q + 1);
+        }
+        const int dd[4] = {d.x, d.y, d.z, d.w};
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            bool pass = dd[j] >= a.dlo && dd[j] <= a.dhi;
+            int key = (int)((k1 >> (8 * j)) & 0xFF) * a.m1 + (int)((k2 >> (8 * j)) & 0xFF) * a.m2 + a.koff;
+            int64_t v0 = (j & 1) ? x[0][j >> 1].y : x[0][j >> 1].x;
+            int64_t v1 = (j & 1) ? x[1][j >> 1].y : x[1][j >> 1].x;
+            int64_t v2 = (j & 1) ? x[2][j >> 1].y : x[2][j >> 1].x;
+            int64_t v3 = (j & 1) ? x[3][j >> 1].y : x[3][j >> 1].x;
+            q1_row<G, NARROW>(A, a, pass, key, v0, v1, v2, v3);
+        }
+    }
+    // ragged tail (n % 4 rows): thread 0 of the grid
+    if (tid == 0) {
+        for (int64_t r = a.nquads * 4; r < a.n; ++r) {
+            int dd = a.d[r];
+            bool pass = dd >= a.dlo && dd <= a.dhi;
+            int key = (int)a.k1[r] * a.m1 + (int)a.k2[r] * a.m2 + a.koff;
+            q1_row<G, NARROW>(A, a, pass, key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
+        }
+    }
+
+    // ---- hierarchical fold: warp (int64, proven) -> CTA (i128) -> grid ----
+    __shared__ i128 s_part[Q1_THREADS / 32][G][6];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+#pragma unroll
+    for (int g = 0; g < G; ++g) {
+        int64_t v[6] = {A.s0[g], A.s1[g], A.s2[g], A.s3[g], A.dc[g] & ((1ll << Q1_CSHIFT) - 1), A.dc[g] >> Q1_CSHIFT};
+#pragma unroll
+        for (int k = 0; k < 6; ++k) {
+            int64_t w = warp_sum_i64(v[k]);
+            if (lane == 0) s_part[warp][g][k] = (i128)w;
+        }
+    }
+    __syncthreads();
+    if (threadIdx.x < G * 6) {
+        const int g = threadIdx.x / 6, k = threadIdx.x % 6;
+        i128 t = 0;
+        for (int w = 0; w < Q1_THREADS / 32; ++w) t += s_part[w][g][k];
+        put_i128(&parts[(size_t)blockIdx.x * G * 6 + threadIdx.x], t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < G * 6) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[threadIdx.x], t);  // [G][6] raw slots, remapped by k_q1_remap
+    }
+}
+
+// Map the Q1 fragment's raw [G][6] sums to the plan's [ngroups][naggs+1].
+struct Q1Map {
+    int32_t naggs, ngroups;
+    int32_t src[VD_MAX_AGGS];  // raw slot (0..5) per plan aggregate
+};
+template <int G>
+__global__ void k_q1_remap(const Slot16* __restrict__ raw, Q1Map m, Slot16* __restrict__ out) {
+    int k = threadIdx.x;
+    int slots = m.ngroups * (m.naggs + 1);
+    if (k >= slots) return;
+    int g = k / (m.naggs + 1), a = k % (m.naggs + 1);
+    int s = (a == m.naggs) ? 5 : m.src[a];
+    out[k] = raw[g * 6 + s];
+}
+
+// ============================================================================
+// Scalar fragment (Q6 / selective aggregation):
+//   filter: up to 3 columns, ints as inclusive intervals, floats as <= 2 terms
+//   value : product of 1 or 2 columns (+ COUNT)
+// ============================================================================
+template <typename F0, typename F1, typename F2, typename VA, typename VB>
+struct ScalarArgs {
+    const F0* f0; const F1* f1; const F2* f2;
+    int64_t lo[3], hi[3];   // integer intervals
+    int32_t fcmp[2];        // float terms on f0 (cmp codes, -1 unused)
+    double fc[2];
+    const VA* va; const VB* vb;
+    int64_t n;
+};
+
+struct NoCol {};
+
+template <typename T> struct AccOf { typedef int64_t type; };
+template <> struct AccOf<float> { typedef double type; };
+template <> struct AccOf<double> { typedef double type; };
+
+template <typename T>
+__device__ __forceinline__ bool ftest(T x, int k, const int64_t* lo, const int64_t* hi, const int32_t* fc,
+                                      const double* fv) {
+    if (IsFloat<T>::value) {
+        if (x != x) return false;
+        bool ok = true;
+        if (fc[0] >= 0) ok = ok && cmp_flt(fc[0], (double)x, fv[0]);
+        if (fc[1] >= 0) ok = ok && cmp_flt(fc[1], (double)x, fv[1]);
+        return ok;
+    }
+    return (int64_t)x >= lo[k] && (int64_t)x <= hi[k];
+}
+
+constexpr int SC_THREADS = 256;
+
+// MODE 0 branching (late loads: a later column is loaded only for rows whose
+// earlier filters passed), MODE 1 predicated (all loads, contribution x p).
+template <int MODE, bool HAS_F1, bool HAS_F2, bool HAS_VB, typename F0, typename F1, typename F2, typename VA,
+          typename VB>
+__global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constant__ ScalarArgs<F0, F1, F2, VA, VB> a,
+                                                            Slot16* __restrict__ parts, unsigned int* __restrict__ done,
+                                                            Slot16* __restrict__ out) {
+    typedef typename AccOf<VA>::type ACC;
+    ACC sum = 0;
+    int64_t cnt = 0;
+    const int64_t nthreads = (int64_t)gridDim.x * SC_THREADS;
+    const int64_t tid = (int64_t)blockIdx.x * SC_THREADS + threadIdx.x;
+    const int64_t nq = a.n / 4;
+    for (int64_t q = tid; q < nq; q += nthreads) {
+        F0 x0[4];
+        {
+            // 4 rows of the first filter column: one 4*sizeof(F0)-byte load
+            if (sizeof(F0) == 4) {
+                int4 t = __ldg(reinterpret_cast<const int4*>(a.f0) + q);
+                memcpy(&x0[0], &t.x, 4); memcpy(&x0[1], &t.y, 4); memcpy(&x0[2], &t.z, 4); memcpy(&x0[3], &t.w, 4);
+            } else if (sizeof(F0) == 8) {
+                longlong2 t0 = __ldg(reinterpret_cast<const longlong2*>(a.f0) + 2 * q);
+                longlong2 t1 = __ldg(reinterpret_cast<const longlong2*>(a.f0) + 2 * q + 1);
+                memcpy(&x0[0], &t0.x, 8); memcpy(&x0[1], &t0.y, 8); memcpy(&x0[2], &t1.x, 8); memcpy(&x0[3], &t1.y, 8);
+            } else {
+#pragma unroll
+                for (int j = 0; j < 4; ++j) x0[j] = a.f0[4 * q + j];
+            }
+        }
+        unsigned p = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) p |= (ftest(x0[j], 0, a.lo, a.hi, a.fcmp, a.fc) ? 1u : 0u) << j;
+        if (MODE == 0 && p == 0) continue;  // late loads: nothing of this quad survives
+        if (HAS_F1) {
+            F1 x1[4];
+#pragma unroll
+            for (int j = 0; j < 4; ++j) x1[j] = (MODE == 1 || ((p >> j) & 1)) ? __ldg(a.f1 + 4 * q + j) : F1(0);
+            unsigned p1 = 0;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) p1 |= (ftest(x1[j], 1, a.lo, a.hi, a.fcmp, a.fc) ? 1u : 0u) << j;
+            p &= p1;
+            if (MODE == 0 && p == 0) continue;
+        }
+        if (HAS_F2) {
+            F2 x2[4];
+#pragma unroll
+            for (int j = 0; j < 4; ++j) x2[j] = (MODE == 1 || ((p >> j) & 1)) ? __ldg(a.f2 + 4 * q + j) : F2(0);
+            unsigned p2 = 0;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) p2 |= (ftest(x2[j], 2, a.lo, a.hi, a.fcmp, a.fc) ? 1u : 0u) << j;
+            p &= p2;
+            if (MODE == 0 && p == 0) continue;
+        }
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            const bool pj = (p >> j) & 1;
+            if (MODE == 0 && !pj) continue;
+            VA va = (a.va == (const VA*)a.f0) ? (VA)x0[j] : __ldg(a.va + 4 * q + j);
+            ACC v = (ACC)va;
+            if (HAS_VB) v *= (ACC)__ldg(a.vb + 4 * q + j);
+            if (MODE == 1) { sum += pj ? v : (ACC)0; cnt += pj; }
+            else { sum += v; cnt += 1; }
+        }
+    }
+    if (tid == 0) {
+        for (int64_t r = nq * 4; r < a.n; ++r) {
+            bool pj = ftest(a.f0[r], 0, a.lo, a.hi, a.fcmp, a.fc);
+            if (HAS_F1) pj = pj && ftest(a.f1[r], 1, a.lo, a.hi, a.fcmp, a.fc);
+            if (HAS_F2) pj = pj && ftest(a.f2[r], 2, a.lo, a.hi, a.fcmp, a.fc);
+            if (!pj) continue;
+            ACC v = (ACC)a.va[r];
+            if (HAS_VB) v *= (ACC)a.vb[r];
+            sum += v;
+            cnt += 1;
+        }
+    }
+    // warp -> CTA -> grid
+    __shared__ Slot16 s_w[SC_THREADS / 32][2];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    int64_t c = warp_sum_i64(cnt);
+    if (IsFloat<VA>::value) {
+        double s = warp_sum_f64((double)sum);
+        if (lane == 0) put_f64(&s_w[warp][0], s);
+    } else {
+        i128 s = warp_sum_i128((i128)(int64_t)sum);
+        if (lane == 0) put_i128(&s_w[warp][0], s);
+    }
+    if (lane == 0) put_i128(&s_w[warp][1], (i128)c);
+    __syncthreads();
+    if (threadIdx.x < 2) {
+        Slot16 r = s_w[0][threadIdx.x];
+        for (int w = 1; w < SC_THREADS / 32; ++w) {
+            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(s_w[w][0]));
+            else put_i128(&r, get_i128(r) + get_i128(s_w[w][threadIdx.x]));
+        }
+        parts[(size_t)blockIdx.x * 2 + threadIdx.x] = r;
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < 2) {
+        Slot16 r;
+        r.lo = __ldcg(&parts[threadIdx.x].lo);
+        r.hi = __ldcg(&parts[threadIdx.x].hi);
+        for (unsigned b = 1; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
+            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
+            else put_i128(&r, get_i128(r) + get_i128(x));
+        }
+        out[threadIdx.x] = r;  // raw [sum, count], remapped by k_scalar_remap
+    }
+}
+
+struct ScalarMap {
+    int32_t naggs;
+    int32_t src[VD_MAX_AGGS];  // 0 = sum, 1 = count
+};
+__global__ void k_scalar_remap(const Slot16* __restrict__ raw, ScalarMap m, Slot16* __restrict__ out) {
+    int k = threadIdx.x;
+    if (k > m.naggs) return;
+    out[k] = raw[(k == m.naggs) ? 1 : m.src[k]];
+}
+
+// ============================================================================
+// Host planner
+// ============================================================================
+struct Bound {
+    bool known;
+    double lo, hi;  // value bounds (doubles: only used for overflow proofs)
+};
+
+static Bound col_bound(const vd_pipeline* p, const vd_column* cols, int ncols, const vd_column* dims, int c) {
+    const vd_column* col = nullptr;
+    if (c < ncols) col = &cols[c];
+    else col = &dims[p->gathers[c - ncols].dim_col];
+    Bound b;
+    b.known = col->has_minmax && col->dtype != VD_F32 && col->dtype != VD_F64;
+    b.lo = (double)col->min;
+    b.hi = (double)col->max;
+    return b;
+}
+
+static double factor_absmax(const vd_factor& f, const Bound& b) {
+    if (f.col < 0) return std::fabs((double)f.a);
+    double x1 = (double)f.a + (double)f.b * b.lo, x2 = (double)f.a + (double)f.b * b.hi;
+    return std::max(std::fabs(x1), std::fabs(x2));
+}
+
+static int col_dtype(const vd_pipeline* p, const vd_column* cols, int ncols, const vd_column* dims, int c) {
+    if (c < ncols) return cols[c].dtype;
+    return dims[p->gathers[c - ncols].dim_col].dtype;
+}
+
+// Fold the conjunction's integer terms on column c into [lo, hi]; false if a
+// term is not an interval (NE / IN) or a float.
+static bool term_interval(const vd_term& t, int64_t* lo, int64_t* hi) {
+    switch (t.cmp) {
+    case VD_CMP_GT: if (t.ival == INT64_MAX) return false; *lo = std::max(*lo, t.ival + 1); return true;
+    case VD_CMP_GE: *lo = std::max(*lo, t.ival); return true;
+    case VD_CMP_LT: if (t.ival == INT64_MIN) return false; *hi = std::min(*hi, t.ival - 1); return true;
+    case VD_CMP_LE: *hi = std::min(*hi, t.ival); return true;
+    case VD_CMP_EQ: *lo = std::max(*lo, t.ival); *hi = std::min(*hi, t.ival); return true;
+    default: return false;
+    }
+}
+
+static int grid_persistent(int per_sm) { return num_sms() * per_sm; }
+
+// ---- Q1 matching ---------------------------------------------------------
+static bool plain_col(const vd_factor& f) { return f.col >= 0 && f.a == 0 && f.b == 1; }
+
+static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, void* out, void* ws,
+                        cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    if (p->ngathers != 0 || p->nkeyparts != 2 || p->ngroups > 8 || p->ngroups < 1) return VD_OK;
+    for (int k = 0; k < 2; ++k) {
+        const vd_keypart& kp = p->key[k];
+        if (kp.col >= ncols || kp.fn != 0 || cols[kp.col].dtype != VD_U8) return VD_OK;
+        if (kp.mult < -1000 || kp.mult > 1000 || kp.sub < -1000 || kp.sub > 1000) return VD_OK;
+        if (!cols[kp.col].has_minmax) return VD_OK;
+    }
+    // key domain proof from metadata (ctrl/data bit conflict check)
+    {
+        double klo = 0, khi = 0;
+        for (int k = 0; k < 2; ++k) {
+            const vd_keypart& kp = p->key[k];
+            double a = ((double)cols[kp.col].min - kp.sub) * kp.mult, b = ((double)cols[kp.col].max - kp.sub) * kp.mult;
+            klo += std::min(a, b);
+            khi += std::max(a, b);
+        }
+        if (klo < 0 || khi >= (double)p->ngroups) return VD_OK;  // generic path counts violations
+    }
+    // predicate: one conjunction over a single i32 column, intervals only
+    int dcol = -1;
+    int64_t lo = INT32_MIN, hi = INT32_MAX;
+    if (p->pred.nconj > 1) return VD_OK;
+    if (p->pred.nconj == 1) {
+        for (int k = 0; k < p->pred.conj[0].nterms; ++k) {
+            const vd_term& t = p->pred.conj[0].terms[k];
+            if (t.col >= ncols || cols[t.col].dtype != VD_I32) return VD_OK;
+            if (dcol >= 0 && t.col != dcol) return VD_OK;
+            dcol = t.col;
+            if (!term_interval(t, &lo, &hi)) return VD_OK;
+        }
+    }
+    if (dcol < 0) return VD_OK;  // need a predicate column for this fragment
+    lo = std::max<int64_t>(lo, INT32_MIN);
+    hi = std::min<int64_t>(hi, INT32_MAX);
+    // aggregates -> raw slots; roles V0..V3
+    int V[4] = {-1, -1, -1, -1};
+    int64_t a1 = 0, b1 = 0, a2 = 0, b2 = 0;
+    bool have_lin1 = false, have_lin2 = false;
+    Q1Map map;
+    map.naggs = p->naggs;
+    map.ngroups = (int32_t)p->ngroups;
+    auto setrole = [&](int r, int c) {
+        if (V[r] >= 0 && V[r] != c) return false;
+        V[r] = c;
+        return true;
+    };
+    // first pass: the product aggregates fix V1, V2, V3
+    for (int k = 0; k < p->naggs; ++k) {
+        const vd_agg& g = p->aggs[k];
+        if (g.kind == VD_AGG_COUNT) { map.src[k] = 5; continue; }
+        if (g.kind != VD_AGG_SUM) return VD_OK;
+        if (g.nfactors < 1 || g.nfactors > 3 || !plain_col(g.f[0])) return VD_OK;
+        for (int f = 0; f < g.nfactors; ++f) {
+            if (g.f[f].col < 0 || g.f[f].col >= ncols || cols[g.f[f].col].dtype != VD_I64) return VD_OK;
+        }
+        if (g.nfactors >= 2) {
+            if (!setrole(1, g.f[0].col) || !setrole(2, g.f[1].col)) return VD_OK;
+            if (have_lin1 && (a1 != g.f[1].a || b1 != g.f[1].b)) return VD_OK;
+            a1 = g.f[1].a; b1 = g.f[1].b; have_lin1 = true;
+            if (g.nfactors == 3) {
+                if (!setrole(3, g.f[2].col)) return VD_OK;
+                if (have_lin2 && (a2 != g.f[2].a || b2 != g.f[2].b)) return VD_OK;
+                a2 = g.f[2].a; b2 = g.f[2].b; have_lin2 = true;
+                map.src[k] = 3;
+            } else {
+                map.src[k] = 2;
+            }
+        }
+    }
+    // second pass: single-column sums take V1 / V2 / V0
+    for (int k = 0; k < p->naggs; ++k) {
+        const vd_agg& g = p->aggs[k];
+        if (g.kind != VD_AGG_SUM || g.nfactors != 1) continue;
+        int c = g.f[0].col;
+        if (V[1] == c) map.src[k] = 1;
+        else if (V[2] == c) map.src[k] = 4;
+        else if (V[0] < 0 || V[0] == c) { V[0] = c; map.src[k] = 0; }
+        else if (V[1] < 0) { V[1] = c; map.src[k] = 1; }
+        else if (V[2] < 0) { V[2] = c; map.src[k] = 4; }
+        else return VD_OK;
+    }
+    // unused roles read some valid column (cheap, keeps one code path)
+    int anycol = -1;
+    for (int r = 0; r < 4; ++r) if (V[r] >= 0) anycol = V[r];
+    if (anycol < 0) anycol = -2;
+    // overflow proof: per-thread int64 over rows_per_thread rows, warp sums too
+    int grid = grid_persistent(2);
+    int64_t threads = (int64_t)grid * Q1_THREADS;
+    double rows_per_warp = std::ceil((double)n / (double)threads) * 32.0 + 64.0;
+    Bound bv[4];
+    for (int r = 0; r < 4; ++r) {
+        int c = V[r] >= 0 ? V[r] : (anycol >= 0 ? anycol : -1);
+        if (c < 0) { bv[r].known = true; bv[r].lo = bv[r].hi = 0; continue; }
+        bv[r] = col_bound(p, cols, ncols, nullptr, c);
+        if (!bv[r].known) return VD_OK;
+    }
+    auto amax = [](const Bound& b) { return std::max(std::fabs(b.lo), std::fabs(b.hi)); };
+    double f1 = std::max(std::fabs((double)a1 + (double)b1 * bv[2].lo), std::fabs((double)a1 + (double)b1 * bv[2].hi));
+    double f2 = std::max(std::fabs((double)a2 + (double)b2 * bv[3].lo), std::fabs((double)a2 + (double)b2 * bv[3].hi));
+    double dpmax = amax(bv[1]) * f1, chmax = dpmax * f2;
+    const double LIM = 9.0e18;
+    if (rows_per_warp * std::max({amax(bv[0]), amax(bv[1]), dpmax, chmax}) >= LIM) return VD_OK;
+    if (amax(bv[2]) * rows_per_warp >= (double)(1ll << Q1_CSHIFT) || bv[2].lo < 0) return VD_OK;
+    if (rows_per_warp >= (double)(1ll << (63 - Q1_CSHIFT))) return VD_OK;
+    auto fits32 = [](int64_t x) { return x > INT32_MIN && x < INT32_MAX; };
+    bool narrow = amax(bv[1]) < 2147483647.0 && f1 < 2147483647.0 && dpmax < 2147483647.0 && f2 < 2147483647.0 &&
+                  amax(bv[2]) < 2147483647.0 && amax(bv[3]) < 2147483647.0 && fits32(a1) && fits32(b1) &&
+                  fits32(a2) && fits32(b2);
+    // alignment for the vector loads
+    auto al = [](const void* q, size_t a) { return ((uintptr_t)q % a) == 0; };
+    if (!al(cols[dcol].data, 16) || !al(cols[p->key[0].col].data, 4) || !al(cols[p->key[1].col].data, 4)) return VD_OK;
+    Q1Args qa;
+    qa.d = (const int32_t*)cols[dcol].data;
+    qa.dlo = (int32_t)lo;
+    qa.dhi = (int32_t)hi;
+    qa.k1 = (const uint8_t*)cols[p->key[0].col].data;
+    qa.k2 = (const uint8_t*)cols[p->key[1].col].data;
+    qa.m1 = (int32_t)p->key[0].mult;
+    qa.m2 = (int32_t)p->key[1].mult;
+    qa.koff = (int32_t)(-p->key[0].sub * p->key[0].mult - p->key[1].sub * p->key[1].mult);
+    for (int r = 0; r < 4; ++r) {
+        int c = V[r] >= 0 ? V[r] : anycol;
+        if (c < 0) return VD_OK;
+        qa.v[r] = (const int64_t*)cols[c].data;
+        if (!al(qa.v[r], 16)) return VD_OK;
+    }
+    qa.a1 = a1; qa.b1 = b1; qa.a2 = a2; qa.b2 = b2;
+    qa.nquads = n / 4;
+    qa.n = n;
+    // workspace: [done (256B)] [parts grid*G*6*16] [raw G*6*16]
+    int G = p->ngroups <= 4 ? 4 : (p->ngroups <= 6 ? 6 : 8);
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    Slot16* raw = parts + (size_t)grid * G * 6;
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+#define Q1_LAUNCH(GG)                                                                                    \
+    if (narrow) k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                     \
+    else k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                           \
+    k_q1_remap<GG><<<1, 1024, 0, s>>>(raw, map, (Slot16*)out);
+    if (G == 4) { Q1_LAUNCH(4) } else if (G == 6) { Q1_LAUNCH(6) } else { Q1_LAUNCH(8) }
+#undef Q1_LAUNCH
+    *nl += 2;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    *done = true;
+    return VD_OK;
+}
+
+// ---- scalar matching ----------------------------------------------------------
+template <int MODE, bool HF1, bool HF2, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+static cudaError_t launch_scalar(const ScalarArgs<F0, F1, F2, VA, VB>& sa, void* ws, Slot16* out, const ScalarMap& m,
+                                 cudaStream_t s, int* nl) {
+    int grid = grid_persistent(4);
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    Slot16* raw = parts + (size_t)grid * 2;
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) return e;
+    k_pipe_scalar<MODE, HF1, HF2, HVB, F0, F1, F2, VA, VB><<<grid, SC_THREADS, 0, s>>>(sa, parts, dn, raw);
+    k_scalar_remap<<<1, 32, 0, s>>>(raw, m, out);
+    *nl += 2;
+    return cudaGetLastError();
+}
+
+static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, void* out, void* ws,
+                            cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    if (p->ngathers != 0 || p->nkeyparts != 0 || p->ngroups != 1) return VD_OK;
+    if (p->pred.nconj != 1) return VD_OK;
+    // filter columns in order of first appearance
+    int fcol[3] = {-1, -1, -1};
+    int nf = 0;
+    int64_t lo[3] = {INT64_MIN, INT64_MIN, INT64_MIN}, hi[3] = {INT64_MAX, INT64_MAX, INT64_MAX};
+    int32_t fcmp[2] = {-1, -1};
+    double fc[2] = {0, 0};
+    int nfl = 0;
+    for (int k = 0; k < p->pred.conj[0].nterms; ++k) {
+        const vd_term& t = p->pred.conj[0].terms[k];
+        if (t.col >= ncols) return VD_OK;
+        int slot = -1;
+        for (int j = 0; j < nf; ++j) if (fcol[j] == t.col) slot = j;
+        if (slot < 0) {
+            if (nf == 3) return VD_OK;
+            slot = nf;
+            fcol[nf++] = t.col;
+        }
+        int dt = cols[t.col].dtype;
+        if (dt == VD_F32 || dt == VD_F64) {
+            if (slot != 0 || nfl == 2 || t.cmp == VD_CMP_IN) return VD_OK;
+            fcmp[nfl] = t.cmp;
+            fc[nfl] = t.fval;
+            ++nfl;
+        } else if (!term_interval(t, &lo[slot], &hi[slot])) {
+            return VD_OK;
+        }
+    }
+    // aggregates: one SUM of 1-2 plain columns, and/or COUNT
+    int va = -1, vb = -1;
+    ScalarMap m;
+    m.naggs = p->naggs;
+    for (int k = 0; k < p->naggs; ++k) {
+        const vd_agg& g = p->aggs[k];
+        if (g.kind == VD_AGG_COUNT) { m.src[k] = 1; continue; }
+        if (g.kind != VD_AGG_SUM || g.nfactors > 2 || va >= 0) return VD_OK;
+        for (int f = 0; f < g.nfactors; ++f) if (!plain_col(g.f[f]) || g.f[f].col >= ncols) return VD_OK;
+        va = g.f[0].col;
+        vb = g.nfactors == 2 ? g.f[1].col : -1;
+        m.src[k] = 0;
+    }
+    if (va < 0) va = fcol[0];
+    if (va < 0) return VD_OK;
+    int t0 = nf > 0 ? cols[fcol[0]].dtype : -1;
+    int t1 = nf > 1 ? cols[fcol[1]].dtype : -1;
+    int t2 = nf > 2 ? cols[fcol[2]].dtype : -1;
+    int tva = cols[va].dtype, tvb = vb >= 0 ? cols[vb].dtype : -1;
+    auto al16 = [](const void* q) { return ((uintptr_t)q % 16) == 0; };
+    int mode = p->sel_mode == VD_SEL_PREDICATED ? 1 : 0;
+    // overflow proof for integer products (per-thread int64, warp in int128)
+    if (tva == VD_I64) {
+        Bound A = col_bound(p, cols, ncols, nullptr, va);
+        Bound B = vb >= 0 ? col_bound(p, cols, ncols, nullptr, vb) : Bound{true, 1, 1};
+        if (!A.known || !B.known) return VD_OK;
+        double mx = std::max(std::fabs(A.lo), std::fabs(A.hi)) * std::max(std::fabs(B.lo), std::fabs(B.hi));
+        double rows = std::ceil((double)n / ((double)grid_persistent(4) * SC_THREADS)) + 8;
+        if (mx * rows >= 9.0e18) return VD_OK;
+    }
+    cudaError_t e = cudaSuccess;
+    Slot16* o = (Slot16*)out;
+    // Q6 shape: filters (i32, i64, i64), value i64 * i64
+    if (nf == 3 && t0 == VD_I32 && t1 == VD_I64 && t2 == VD_I64 && tva == VD_I64 && tvb == VD_I64 &&
+        al16(cols[fcol[0]].data)) {
+        ScalarArgs<int32_t, int64_t, int64_t, int64_t, int64_t> sa;
+        sa.f0 = (const int32_t*)cols[fcol[0]].data;
+        sa.f1 = (const int64_t*)cols[fcol[1]].data;
+        sa.f2 = (const int64_t*)cols[fcol[2]].data;
+        for (int j = 0; j < 3; ++j) { sa.lo[j] = lo[j]; sa.hi[j] = hi[j]; }
+        sa.fcmp[0] = sa.fcmp[1] = -1;
+        sa.fc[0] = sa.fc[1] = 0;
+        sa.va = (const int64_t*)cols[va].data;
+        sa.vb = (const int64_t*)cols[vb].data;
+        sa.n = n;
+        if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
+        else e = launch_scalar<0, true, true, true>(sa, ws, o, m, s, nl);
+    } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && al16(cols[fcol[0]].data)) {
+        // selective aggregation over one f32 column (Fig 15 / C1)
+        ScalarArgs<float, float, float, float, float> sa;
+        sa.f0 = (const float*)cols[fcol[0]].data;
+        sa.f1 = sa.f2 = nullptr;
+        for (int j = 0; j < 3; ++j) { sa.lo[j] = lo[j]; sa.hi[j] = hi[j]; }
+        sa.fcmp[0] = fcmp[0]; sa.fcmp[1] = fcmp[1];
+        sa.fc[0] = fc[0]; sa.fc[1] = fc[1];
+        sa.va = (const float*)cols[va].data;
+        sa.vb = nullptr;
+        sa.n = n;
+        if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
+        else e = launch_scalar<0, false, false, false>(sa, ws, o, m, s, nl);
+    } else {
+        return VD_OK;
+    }
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    *done = true;
+    return VD_OK;
+}
+
+// ---- generic -------------------------------------------------------------------
+static size_t gen_smem(const vd_pipeline* p, bool smem_acc) {
+    size_t nslots = (size_t)p->ngroups * (p->naggs + 1);
+    size_t b = (size_t)GEN_WARPS * 32 * (p->naggs + 1) * sizeof(Slot16);
+    if (smem_acc) b += (size_t)GEN_WARPS * nslots * sizeof(Slot16);
+    return b;
+}
+static const size_t GEN_SMEM_MAX = 200 * 1024;
+
+size_t pipeline_ws_bytes(const vd_pipeline* p) {
+    size_t nslots = (size_t)p->ngroups * (p->naggs + 1);
+    size_t grid = (size_t)grid_persistent(4);
+    size_t gen = 256 + grid * nslots * sizeof(Slot16) + 2 * nslots * sizeof(Slot16) + 256;
+    size_t q1 = 256 + grid * 8 * 6 * sizeof(Slot16) + 8 * 6 * sizeof(Slot16);
+    size_t sc = 256 + grid * 2 * sizeof(Slot16) + 2 * sizeof(Slot16);
+    size_t b = std::max(gen, std::max(q1, sc)) + 256;
+    return (b + 255) & ~(size_t)255;
+}
+
+static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                             void* out, void* ws, cudaStream_t s, int* nl) {
+    GenPlan P;
+    std::memset(&P, 0, sizeof(P));
+    make_devpred(&p->pred, &P.pred);
+    P.cols.ncols = ncols;
+    for (int c = 0; c < ncols; ++c) { P.cols.p[c] = cols[c].data; P.cols.dt[c] = cols[c].dtype; }
+    P.ngathers = p->ngathers;
+    for (int g = 0; g < p->ngathers; ++g) {
+        P.g_fk[g] = p->gathers[g].fk_col;
+        P.g_bias[g] = p->gathers[g].bias;
+        const vd_column& d = dims[p->gathers[g].dim_col];
+        P.g_p[g] = d.data;
+        P.g_len[g] = d.len;
+        P.g_dt[g] = d.dtype;
+    }
+    P.nkey = p->nkeyparts;
+    for (int k = 0; k < p->nkeyparts; ++k) {
+        P.k_col[k] = p->key[k].col;
+        P.k_fn[k] = p->key[k].fn;
+        P.k_sub[k] = p->key[k].sub;
+        P.k_mult[k] = p->key[k].mult;
+    }
+    P.ngroups = p->ngroups;
+    P.naggs = p->naggs;
+    for (int a = 0; a < p->naggs; ++a) {
+        const vd_agg& g = p->aggs[a];
+        P.agg[a].kind = g.kind;
+        P.agg[a].nf = g.nfactors;
+        bool isf = false;
+        for (int f = 0; f < g.nfactors; ++f) {
+            P.agg[a].col[f] = g.f[f].col;
+            P.agg[a].a[f] = g.f[f].a;
+            P.agg[a].b[f] = g.f[f].b;
+            if (g.kind != VD_AGG_COUNT && g.f[f].col >= 0) {
+                int dt = col_dtype(p, cols, ncols, dims, g.f[f].col);
+                isf = isf || dt == VD_F32 || dt == VD_F64;
+            }
+        }
+        P.agg[a].isf = isf;
+    }
+    const int nslots = (int)(p->ngroups * (p->naggs + 1));
+    bool smem_acc = gen_smem(p, true) <= GEN_SMEM_MAX;
+    size_t smem = gen_smem(p, smem_acc);
+    int grid = grid_persistent(smem_acc && smem > 100 * 1024 ? 1 : 2);
+    int64_t maxg = (n + GEN_THREADS - 1) / GEN_THREADS;
+    if (maxg < 1) maxg = 1;
+    if (grid > maxg) grid = (int)maxg;
+    unsigned int* dn = (unsigned int*)ws;
+    unsigned long long* derr = (unsigned long long*)((char*)ws + 128);
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    Slot16* gacc = parts;  // (global-atomic variant) accumulators
+    unsigned long long* gmask = (unsigned long long*)(gacc + nslots);
+    cudaError_t e = cudaMemsetAsync(ws, 0, 256, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    if (smem_acc) {
+        if (smem > 48 * 1024) cudaFuncSetAttribute(k_pipe_generic<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_generic<true><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn, (Slot16*)out, derr);
+    } else {
+        // global accumulators: zero sums, +/- extremes for min/max images
+        e = cudaMemsetAsync(gacc, 0, (size_t)nslots * sizeof(Slot16) + (size_t)nslots * 8, s);
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+        bool any_mm = false;
+        for (int a = 0; a < p->naggs; ++a) any_mm |= (p->aggs[a].kind == VD_AGG_MIN || p->aggs[a].kind == VD_AGG_MAX);
+        if (any_mm) { set_error("MIN/MAX with more groups than fit in shared memory"); return VD_E_UNSUPPORTED; }
+        if (smem > 48 * 1024) cudaFuncSetAttribute(k_pipe_generic<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_generic<false><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn, (Slot16*)out, derr);
+    }
+    ++*nl;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    return VD_OK;
+}
+
+vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncols, int64_t n, const vd_column* dims,
+                       int32_t, void* out, void* ws, size_t, cudaStream_t s, int* nl) {
+    if (n == 0) {
+        cudaError_t e = cudaMemsetAsync(out, 0, (size_t)p->ngroups * (p->naggs + 1) * 16, s);
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+        return VD_OK;
+    }
+    if (!p->force_generic) {
+        bool done = false;
+        vd_status st = try_q1(p, cols, ncols, n, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+        st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+    }
+    return run_generic(p, cols, ncols, n, dims, out, ws, s, nl);
+}
+
+}  // namespace vd

@@ -1,0 +1,159 @@
+// vd_common.cuh -- device helpers shared by the libvd kernels (sm_100a).
+// Product code: nothing here is shared with oracle/.
+#pragma once
+
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include "vd.h"
+
+typedef __int128 i128;
+typedef unsigned __int128 u128;
+
+#define VD_FULL 0xFFFFFFFFu
+
+namespace vd {
+
+// ---- empty-slot sentinels (include/vd.h "Empty slots") -------------------
+template <typename T> struct Eps;
+template <> struct Eps<uint8_t> {
+    static __host__ __device__ __forceinline__ bool is(uint8_t v) { return v == 0xFF; }
+    static __host__ __device__ __forceinline__ uint8_t value() { return 0xFF; }
+};
+template <> struct Eps<int32_t> {
+    static __host__ __device__ __forceinline__ bool is(int32_t v) { return v == INT32_MIN; }
+    static __host__ __device__ __forceinline__ int32_t value() { return INT32_MIN; }
+};
+template <> struct Eps<int64_t> {
+    static __host__ __device__ __forceinline__ bool is(int64_t v) { return v == INT64_MIN; }
+    static __host__ __device__ __forceinline__ int64_t value() { return INT64_MIN; }
+};
+template <> struct Eps<float> {
+    static __host__ __device__ __forceinline__ bool is(float v) { return v != v; }
+    static __device__ __forceinline__ float value() { return __int_as_float(0x7fc00000); }
+};
+template <> struct Eps<double> {
+    static __host__ __device__ __forceinline__ bool is(double v) { return v != v; }
+    static __device__ __forceinline__ double value() { return __longlong_as_double(0x7ff8000000000000ll); }
+};
+
+template <typename T> struct IsFloat { static constexpr bool value = false; };
+template <> struct IsFloat<float> { static constexpr bool value = true; };
+template <> struct IsFloat<double> { static constexpr bool value = true; };
+
+// ---- loads ---------------------------------------------------------------
+// Read-only path, allocating in L1 (neighbouring lanes' sectors are reused
+// by the sibling vector loads of a thread).
+template <typename T> __device__ __forceinline__ T ldg(const T* p) { return __ldg(p); }
+template <> __device__ __forceinline__ uint8_t ldg<uint8_t>(const uint8_t* p) { return __ldg(p); }
+
+// Streaming 16-byte load that does not allocate in L1 (single-use data).
+__device__ __forceinline__ int4 ld_stream16(const void* p) {
+    int4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v4.s32 {%0,%1,%2,%3}, [%4];"
+                 : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w)
+                 : "l"(p));
+    return r;
+}
+__device__ __forceinline__ int2 ld_stream8(const void* p) {
+    int2 r;
+    asm volatile("ld.global.nc.L1::no_allocate.v2.s32 {%0,%1}, [%2];" : "=r"(r.x), "=r"(r.y) : "l"(p));
+    return r;
+}
+__device__ __forceinline__ int ld_stream4(const void* p) {
+    int r;
+    asm volatile("ld.global.nc.L1::no_allocate.s32 %0, [%1];" : "=r"(r) : "l"(p));
+    return r;
+}
+
+// ---- gpu-scope acquire/release on 64-bit status words ---------------------
+__device__ __forceinline__ uint64_t ld_acquire_u64(const uint64_t* p) {
+    uint64_t v;
+    asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ void st_release_u64(uint64_t* p, uint64_t v) {
+    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(p), "l"(v) : "memory");
+}
+__device__ __forceinline__ uint64_t ld_relaxed_u64(const uint64_t* p) {
+    uint64_t v;
+    asm volatile("ld.relaxed.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");
+    return v;
+}
+
+// ---- warp reductions -------------------------------------------------------
+__device__ __forceinline__ int64_t warp_sum_i64(int64_t v) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(VD_FULL, v, o);
+    return v;
+}
+__device__ __forceinline__ double warp_sum_f64(double v) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v += __shfl_xor_sync(VD_FULL, v, o);
+    return v;
+}
+__device__ __forceinline__ i128 shfl_xor_i128(i128 v, int o) {
+    uint64_t lo = (uint64_t)(u128)v, hi = (uint64_t)((u128)v >> 64);
+    lo = __shfl_xor_sync(VD_FULL, lo, o);
+    hi = __shfl_xor_sync(VD_FULL, hi, o);
+    return (i128)(((u128)hi << 64) | lo);
+}
+__device__ __forceinline__ i128 warp_sum_i128(i128 v) {
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) v += shfl_xor_i128(v, o);
+    return v;
+}
+
+__device__ __forceinline__ unsigned lanemask_lt() {
+    unsigned m;
+    asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m));
+    return m;
+}
+
+// ---- 128-bit global accumulation via 64-bit atomics ----------------------
+// Adds a signed 64-bit value into a little-endian two's-complement 128-bit
+// integer {lo, hi}: the carry out of the low word is derived from the value
+// the atomic returned, so the high word receives every carry exactly and
+// the final sum is independent of the order of the adds.
+__device__ __forceinline__ void atomic_add_i128_i64(unsigned long long* p, int64_t v) {
+    unsigned long long add = (unsigned long long)v;
+    unsigned long long old = atomicAdd(p, add);
+    unsigned long long carry = (old + add) < old ? 1ull : 0ull;
+    unsigned long long hi = (v < 0 ? ~0ull : 0ull) + carry;
+    if (hi) atomicAdd(p + 1, hi);
+}
+__device__ __forceinline__ void atomic_add_i128(unsigned long long* p, i128 v) {
+    unsigned long long lo = (unsigned long long)(u128)v;
+    unsigned long long hi = (unsigned long long)((u128)v >> 64);
+    unsigned long long old = atomicAdd(p, lo);
+    unsigned long long carry = (old + lo) < old ? 1ull : 0ull;
+    hi += carry;
+    if (hi) atomicAdd(p + 1, hi);
+}
+
+__device__ __forceinline__ void st_i128(void* p, i128 v) {
+    uint64_t* q = (uint64_t*)p;
+    q[0] = (uint64_t)(u128)v;
+    q[1] = (uint64_t)((u128)v >> 64);
+}
+__device__ __forceinline__ i128 ld_i128(const void* p) {
+    const uint64_t* q = (const uint64_t*)p;
+    return (i128)(((u128)q[1] << 64) | q[0]);
+}
+
+// ---- calendar year of a day number (days since 1970-01-01) ---------------
+// Civil-from-days in integer arithmetic (proleptic Gregorian), valid for
+// all int32 day numbers >= -719468.
+__host__ __device__ __forceinline__ int32_t year_of_day(int32_t z) {
+    z += 719468;
+    int32_t era = (z >= 0 ? z : z - 146096) / 146097;
+    int32_t doe = z - era * 146097;
+    int32_t yoe = (doe - doe / 1460 + doe / 36524 - doe / 146096) / 365;
+    int32_t y = yoe + era * 400;
+    int32_t doy = doe - (365 * yoe + yoe / 4 - yoe / 100);
+    int32_t mp = (5 * doy + 2) / 153;
+    int32_t m = mp < 10 ? mp + 3 : mp - 9;
+    return y + (m <= 2 ? 1 : 0);
+}
+
+}  // namespace vd

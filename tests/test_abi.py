@@ -1,0 +1,149 @@
+"""CPU checks of the C-ABI boundary: libvd.so loads, exports every function
+include/vd.h declares, its structs match the binding, and the host-only
+logic (control-vector run counting, workspace sizing, argument validation,
+the cross-device merge) behaves.  No kernel is launched here."""
+import ctypes
+import os
+import re
+import struct
+
+import pytest
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def declared_functions():
+    src = open(os.path.join(ROOT, "include", "vd.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    names = set(re.findall(r"^\s*(?:const\s+)?(?:vd_status|size_t|int32_t|const char\*|void)\s*\*?\s*(vd_\w+)\s*\(",
+                           src, flags=re.M))
+    return sorted(names)
+
+
+def test_header_declares_the_north_star_calls():
+    names = declared_functions()
+    for want in ["vd_load_column", "vd_select_branch", "vd_select_predicated", "vd_gather", "vd_scatter",
+                 "vd_fold_sum", "vd_fold_count", "vd_fold_min", "vd_fold_max", "vd_fold_select", "vd_run_pipeline",
+                 "vd_merge_partials", "vd_workspace_bytes", "vd_partition"]:
+        assert want in names
+
+
+def test_library_exports_every_declared_symbol():
+    lib = ctypes.CDLL(os.path.join(ROOT, "paper_journals_pvldb_pirkmzm16_b200", "libvd.so"))
+    missing = [n for n in declared_functions() if not hasattr(lib, n)]
+    assert missing == []
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    assert set(declared_functions()) == set(vd.EXPORTS)
+
+
+def test_struct_layout_matches_binding():
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    vd._check_abi()
+    assert ctypes.sizeof(vd.vd_column) == 48
+    assert vd.version().startswith("voodoo-b200")
+
+
+def test_ctrl_run_counts_reading_A2():
+    """Run metadata: Divide(Range, R) -> runs of R; Modulo with
+    cap 1 or step 0 -> one run; integer step k -> runs of 1 unless cap | k."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    assert vd.ctrl_runs(None, 10) == 1
+    assert vd.ctrl_runs(None, 0) == 0
+    assert vd.ctrl_runs(vd.ctrl(0, 1, 4), 10) == 3
+    assert vd.ctrl_runs(vd.ctrl(0, 1, 4, cap=2), 10) == 3
+    assert vd.ctrl_runs(vd.ctrl(0, 0, 1), 10) == 1
+    assert vd.ctrl_runs(vd.ctrl(0, 1, 1, cap=1), 10) == 1
+    assert vd.ctrl_runs(vd.ctrl(0, 2, 1, cap=2), 10) == 1
+    assert vd.ctrl_runs(vd.ctrl(0, 2, 1, cap=3), 10) == 10
+    assert vd.ctrl_runs(vd.ctrl(0, 1, 100), 10) == 1
+    with pytest.raises(vd.VdError):
+        vd.ctrl_runs(vd.ctrl(0, 2, 3), 10)  # irregular runs: data dependent (device count)
+    with pytest.raises(vd.VdError):
+        vd.ctrl_runs(vd.ctrl(0, 1, 0), 10)  # den 0
+
+
+def test_workspace_sizes_grow_and_validate():
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+    a = vd.workspace_bytes(vd.VD_OP_SELECT, 1000)
+    b = vd.workspace_bytes(vd.VD_OP_SELECT, 10**8)
+    assert 0 < a < b
+    assert vd.workspace_bytes(vd.VD_OP_FOLD, 10**6, vd.ctrl(0, 2, 3)) > vd.workspace_bytes(vd.VD_OP_FOLD, 10**6)
+    assert vd.workspace_bytes(vd.VD_OP_PIPELINE, 10**6, None, plans.q1()) > 0
+    assert vd.partials_bytes(plans.q1()) == 6 * 7 * 16
+
+
+def test_validation_errors_are_synchronous():
+    """Argument errors come back before any launch (include/vd.h 'Errors')."""
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+    plan = plans.q1()
+    c = vd.vd_column()
+    c.dtype, c.len = vd.VD_I32, 10
+    cols = (vd.vd_column * 7)(*([c] * 7))
+    st = vd._L.vd_run_pipeline(ctypes.byref(plan), cols, 7, 10, None, 0, None, None, 0, None)
+    assert st == vd.VD_E_NULL
+    # key domain proof from metadata: rf in [0, 9] cannot fit 6 groups -> VD_E_DOMAIN
+    cs = []
+    for k, dt in enumerate([vd.VD_I32, vd.VD_U8, vd.VD_U8, vd.VD_I64, vd.VD_I64, vd.VD_I64, vd.VD_I64]):
+        x = vd.vd_column()
+        x.data, x.len, x.dtype = 4096, 10, dt
+        if k in (1, 2):
+            x.min, x.max, x.has_minmax = 0, 9, 1
+        cs.append(x)
+    arr = (vd.vd_column * 7)(*cs)
+    st = vd._L.vd_run_pipeline(ctypes.byref(plan), arr, 7, 10, None, 0, ctypes.c_void_p(4096),
+                               ctypes.c_void_p(4096), 1 << 30, None)
+    assert st == vd.VD_E_DOMAIN
+    bad = vd.pipeline(ngroups=0)
+    assert vd._L.vd_run_pipeline(ctypes.byref(bad), arr, 7, 10, None, 0, ctypes.c_void_p(1), ctypes.c_void_p(1),
+                                 1 << 30, None) == vd.VD_E_ARG
+
+
+def test_no_cpu_fallback_without_device():
+    """Compute entry points refuse to run without a CUDA device."""
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    c = vd.vd_column()
+    c.data, c.len, c.dtype = 4096, 4, vd.VD_I64
+    out = ctypes.c_void_p(8192)
+    st = vd._L.vd_fold_sum(ctypes.byref(c), None, out, None, None, ctypes.c_void_p(4096), 1 << 20, None)
+    assert st == vd.VD_E_CUDA
+    assert "no CPU fallback" in vd._L.vd_last_error().decode()
+
+
+def _pack(vals):
+    b = b""
+    for v in vals:
+        if isinstance(v, float):
+            b += struct.pack("<dq", v, 0)
+        else:
+            b += struct.pack("<Qq", v & (2**64 - 1), v >> 64)
+    return b
+
+
+def test_merge_partials_rank_order_int128_and_empty_groups():
+    """Cross-GPU step of the hierarchical fold (Fig 3 one level up): 128-bit
+    sums, min/max over non-empty ranks, empty groups stay empty."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    plan = vd.pipeline(key=[(0, 0, 0, 1)], ngroups=3,
+                       aggs=[("sum", [1]), ("min", [1]), ("max", [1]), ("count",)])
+    c0 = vd.vd_column()
+    c0.dtype = vd.VD_U8
+    c1 = vd.vd_column()
+    c1.dtype = vd.VD_I64
+    big = 2**63 - 1
+    r0 = _pack([big, 5, 9, 2, 2] + [0, 0, 0, 0, 0] + [7, -3, -3, 1, 1])
+    r1 = _pack([big, 1, 4, 3, 3] + [0, 0, 0, 0, 0] + [0, 0, 0, 0, 0])
+    merged = vd.merge_partials(plan, [c0, c1], [], [r0, r1])
+    res = vd.decode_partials(merged, plan)
+    assert res == {0: [2 * big, 1, 9, 5, 5], 2: [7, -3, -3, 1, 1]}
+
+
+def test_pipeline_descriptor_round_trip():
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+    p = plans.q1()
+    assert p.naggs == 6 and p.ngroups == 6 and p.nkeyparts == 2
+    assert p.pred.conj[0].terms[0].cmp == vd.VD_CMP_LE and p.pred.conj[0].terms[0].ival == 10471
+    q = vd.pred([[(0, "in", [0, 3, 63])]])
+    assert q.conj[0].terms[0].ival == (1 | 8 | (1 << 63)) - (1 << 64)

@@ -112,7 +112,8 @@ def test_fig1_branching_equals_predicated_positions():
     v = rng.random(5000).astype(np.float32)
     for t in [0.0, 0.01, 0.5, 0.99, 1.0]:
         t = float(np.float32(t))  # the predicate constant is an f32 (reading A20)
-        p = oracle.run("value := Greater(%r, v.val)\npos := FoldSelect(value)" % t, v__val=v)
+        # hex literal: the oracle parses the exact f32 value
+        p = oracle.run("value := Greater(%s, v.val)\npos := FoldSelect(value)" % t.hex(), v__val=v)
         got = [x for x in p.get("pos") if x is not None]
         # branch-free cursor arithmetic (Ross): write every input, advance by predicate
         out = np.empty(v.size + 1, dtype=np.int64)

@@ -91,7 +91,7 @@ def test_select_sum_interpreter_bruteforce(intent):
     assert pos.tolist() == np.flatnonzero(v < np.float32(t)).tolist()
     p = oracle.Program()
     p.set("input.val", v)
-    p.run(programs.SELECT_SUM.format(intent=intent, t=repr(t)))
+    p.run(programs.SELECT_SUM.format(intent=intent, t=t.hex()))
     assert p.get("count")[0] == c
     got = p.get_float_exact("totalSum")
     assert got[0][0] + got[1][0] == pytest.approx(sh + sl, rel=1e-15)
