@@ -44,7 +44,7 @@ def parse():
     ap.add_argument("--steps", type=int, default=None)
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
-    ap.add_argument("--workload", default="q1", choices=["q1", "q6", "select", "q19", "q9"])
+    ap.add_argument("--workload", default="q1", choices=["q1", "q6", "select", "selpos", "q19", "q9"])
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
     ap.add_argument("--sel-mode", default="branch", choices=["branch", "predicated"])
     ap.add_argument("--selectivity", type=float, default=0.5, help="select workload: fraction selected")
@@ -58,7 +58,7 @@ def parse():
 
 
 def default_sf(w):
-    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0}[w]
+    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0}[w]
 
 
 # ---------------------------------------------------------------------------
@@ -197,6 +197,8 @@ def main():
 
     if args.impl == "reference":
         return reference_arm(args, rank, world, sf)
+    if args.workload == "selpos":
+        return selpos_main(args, rank, world, local)
 
     import torch
     import torch.distributed as dist
@@ -372,6 +374,79 @@ def main():
         print(json.dumps(line), flush=True)
     if world > 1:
         dist.barrier()
+        dist.destroy_process_group()
+
+
+def selpos_main(args, rank, world, local):
+    """C2 (Fig 1 sweep point): select v < t over 1e9 f32 -> int32 positions,
+    branching or predicated (vd_select_*).  Algorithmic bytes: 4 B/row read +
+    4 B per selected row written."""
+    import numpy as np
+    import torch
+    import torch.distributed as dist
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=dev)
+    stream = torch.cuda.current_stream()
+    n_total = args.rows or 10**9
+    a, b = rank * n_total // world, (rank + 1) * n_total // world
+    n = b - a
+    v = torch.empty(n, dtype=torch.float32, device=dev)
+    gen.device(gen.F32_UNIFORM, v.data_ptr(), n, a, seed=args.seed, stream=stream.cuda_stream)
+    t = float(np.float32(args.selectivity))
+    pos = torch.empty(n, dtype=torch.int32, device=dev)
+    cnt = torch.zeros(1, dtype=torch.int64, device=dev)
+    ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_SELECT, n), dev)
+    fn = vd.select_predicated if args.sel_mode == "predicated" else vd.select_branch
+    cols = [vd.column(v)]
+    p = vd.pred([[(0, "<", t)]])
+
+    def step():
+        fn(cols, n, p, out_pos=pos, out_count=cnt, ws=ws, stream=stream)
+
+    for _ in range(max(args.warmup, 3)):
+        step()
+    lps = vd.last_launch_count()
+    torch.cuda.synchronize()
+    steps = args.steps or 200
+    clocks = ClockSampler(local)
+    clocks.start()
+    time.sleep(0.3)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(steps)]
+    for i in range(steps):
+        ev[i][0].record(stream)
+        step()
+        ev[i][1].record(stream)
+    torch.cuda.synchronize()
+    clk = clocks.stop()
+    ms = sum(s.elapsed_time(e) for s, e in ev) / steps
+    if world > 1:
+        tt = torch.tensor([ms], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        ms = float(tt[0])
+    c = int(cnt.item())
+    peak, kind = hbm_peak()
+    alg = (4 * n + 4 * c) / (ms * 1e-3) / 1e9
+    line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "f32", "data": "synthetic (f32 U[0,1), gen/vd_gen.h)",
+            "config": {"workload": f"selpos_f32_{n_total}_s{args.selectivity:g}", "sel_mode": args.sel_mode,
+                       "selected": c, "achieved_selectivity": c / n,
+                       "l2": f"input {4 * n / 1e9:.1f} GB > 126 MB L2: no flush needed"},
+            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
+                         "peak_kind": kind, "traffic": None, "kernel": "k_select", "kernel_ms": ms},
+            "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    if world > 1:
         dist.destroy_process_group()
 
 

@@ -185,6 +185,7 @@ __global__ void __launch_bounds__(FOLD_THREADS) k_fold_seg(const T* __restrict__
     __shared__ int64_t s_first_rid;
     __shared__ int s_first_head;
     __shared__ int s_heads[FOLD_THREADS];
+    __shared__ int64_t s_hrid[FOLD_THREADS];
     const int t = threadIdx.x;
     const int64_t tile = blockIdx.x;
     const int64_t a0 = tile * FOLD_TILE;
@@ -266,6 +267,7 @@ __global__ void __launch_bounds__(FOLD_THREADS) k_fold_seg(const T* __restrict__
         }
         cur.add(x[j]);
     }
+    s_hrid[t] = head_rid;
     // CTA segmented scan of (tail rid, tail agg, cont)
     SegElem<T, OP> me;
     me.rid = cur_rid;
@@ -296,6 +298,17 @@ __global__ void __launch_bounds__(FOLD_THREADS) k_fold_seg(const T* __restrict__
             rec_first[tile] = r;
         } else {
             store_result<T, OP>(out, counts, head_rid, h);
+        }
+    }
+    if (t < FOLD_THREADS - 1 && s_hrid[t + 1] != cur_rid) {
+        // this thread's tail run ends exactly at the thread boundary
+        SegElem<T, OP> tot = s_scan[pb][t];  // inclusive: the run's in-tile aggregate
+        if (cur_rid == first_rid) {
+            SegRec<T, OP> r;
+            r.rid = cur_rid; r.valid = 1; r.starts = first_head; r.single = 0; r.a = tot.a;
+            rec_first[tile] = r;
+        } else {
+            store_result<T, OP>(out, counts, cur_rid, tot.a);
         }
     }
     if (t == FOLD_THREADS - 1) {

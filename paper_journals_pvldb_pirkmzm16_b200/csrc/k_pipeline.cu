@@ -25,6 +25,7 @@
 
 #include <algorithm>
 #include <cmath>
+#include <cstdlib>
 #include <cstring>
 
 #include "vd_common.cuh"
@@ -516,6 +517,179 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
     }
 }
 
+// ---- Q1 fragment, TMA-staged --------------------------------------------------
+// The same fragment with its column tiles staged in shared memory by 1D TMA
+// bulk copies (cp.async.bulk -> UBLKCP): one producer warp keeps
+// Q1T_STAGES tiles of Q1T_TILE rows (7 column slices each) in flight behind
+// mbarriers while eight consumer warps fold the previous tiles out of shared
+// memory.  Group accumulators live in shared memory, one private set per
+// thread laid out [slot][word][thread] (conflict-free: a lane's address
+// depends on the slot only through multiples of 32 banks), so a row's
+// contribution is one address computation plus load-add-store per word with
+// no branch and no per-slot predication; rows failing the predicate land in
+// a trash slot G.  This is the virtual scatter of §3.1.3: the group key is a
+// work-item-local scatter position that is never materialised.
+constexpr int Q1T_CW = 8;                                // consumer warps
+constexpr int Q1T_NT = Q1T_CW * 32;                      // consumer threads
+constexpr int Q1T_THREADS = Q1T_NT + 32;                 // + 1 producer warp
+constexpr int Q1T_TILE = Q1T_CW * 128;                   // rows per stage
+constexpr int Q1T_STAGES = 3;
+constexpr int Q1T_STAGE_BYTES = Q1T_TILE * (4 + 4 * 8 + 2);
+constexpr int Q1T_WORDS = 5;                             // qty, ext, dp, ch, disc|count
+__host__ __device__ constexpr size_t q1t_smem(int G) {
+    return (size_t)Q1T_STAGES * Q1T_STAGE_BYTES + (size_t)(G + 1) * Q1T_WORDS * Q1T_NT * 8 + 2 * Q1T_STAGES * 8;
+}
+
+template <bool NARROW>
+__device__ __forceinline__ void q1_row_smem(int64_t* __restrict__ acc_t, const Q1Args& a, int G, int32_t dd,
+                                            int key, int64_t v0, int64_t v1, int64_t v2, int64_t v3) {
+    const bool pass = dd >= a.dlo && dd <= a.dhi;
+    const int kk = pass ? key : G;  // trash slot for rows that fail the predicate
+    int64_t dp, ch;
+    if (NARROW) {
+        int32_t f1 = (int32_t)a.a1 + (int32_t)a.b1 * (int32_t)v2;
+        dp = (int64_t)(int32_t)v1 * (int64_t)f1;
+        int32_t f2 = (int32_t)a.a2 + (int32_t)a.b2 * (int32_t)v3;
+        ch = (int64_t)(int32_t)dp * (int64_t)f2;
+    } else {
+        dp = v1 * (a.a1 + a.b1 * v2);
+        ch = dp * (a.a2 + a.b2 * v3);
+    }
+    int64_t* p = acc_t + (size_t)kk * Q1T_WORDS * Q1T_NT;
+    p[0 * Q1T_NT] += v0;
+    p[1 * Q1T_NT] += v1;
+    p[2 * Q1T_NT] += dp;
+    p[3 * Q1T_NT] += ch;
+    p[4 * Q1T_NT] += v2 + (1ll << Q1_CSHIFT);
+}
+
+template <int G, bool NARROW>
+__global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_constant__ Q1Args a, int64_t ntiles,
+                                                                Slot16* __restrict__ parts,
+                                                                unsigned int* __restrict__ done,
+                                                                Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    int64_t* acc = reinterpret_cast<int64_t*>(smem + (size_t)Q1T_STAGES * Q1T_STAGE_BYTES);
+    uint64_t* full = reinterpret_cast<uint64_t*>(acc + (size_t)(G + 1) * Q1T_WORDS * Q1T_NT);
+    uint64_t* empty = full + Q1T_STAGES;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < Q1T_STAGES; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], Q1T_NT);
+        }
+        fence_mbar_init();
+    }
+    for (int k = threadIdx.x; k < (G + 1) * Q1T_WORDS * Q1T_NT; k += Q1T_THREADS) acc[k] = 0;
+    __syncthreads();
+
+    if (warp == Q1T_CW) {
+        // ---- producer: one elected lane issues the bulk copies ----
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % Q1T_STAGES);
+                if (it >= Q1T_STAGES) mbar_wait(&empty[s], (uint32_t)(((it / Q1T_STAGES) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * Q1T_STAGE_BYTES;
+                const int64_t r0 = tile * Q1T_TILE;
+                mbar_expect_tx(&full[s], Q1T_STAGE_BYTES);
+                tma_load_1d(st, a.d + r0, Q1T_TILE * 4, &full[s], pol);
+#pragma unroll
+                for (int c = 0; c < 4; ++c)
+                    tma_load_1d(st + Q1T_TILE * 4 + c * Q1T_TILE * 8, a.v[c] + r0, Q1T_TILE * 8, &full[s], pol);
+                tma_load_1d(st + Q1T_TILE * 36, a.k1 + r0, Q1T_TILE, &full[s], pol);
+                tma_load_1d(st + Q1T_TILE * 37, a.k2 + r0, Q1T_TILE, &full[s], pol);
+            }
+        }
+        __syncwarp();  // reconverge the producer warp before the CTA barrier
+    } else {
+        // ---- consumers: warp w folds rows w*128 + {2l, 2l+1, 64+2l, 65+2l} ----
+        int64_t* acc_t = acc + threadIdx.x;
+        const int rb = warp * 128 + 2 * lane;
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % Q1T_STAGES);
+            mbar_wait(&full[s], (uint32_t)((it / Q1T_STAGES) & 1));
+            const uint8_t* st = smem + (size_t)s * Q1T_STAGE_BYTES;
+            int2 dd[2];
+            uint32_t kk1[2], kk2[2];
+            longlong2 x[2][4];
+#pragma unroll
+            for (int h = 0; h < 2; ++h) {
+                const int r = rb + 64 * h;
+                dd[h] = *reinterpret_cast<const int2*>(st + r * 4);
+                kk1[h] = *reinterpret_cast<const uint16_t*>(st + Q1T_TILE * 36 + r);
+                kk2[h] = *reinterpret_cast<const uint16_t*>(st + Q1T_TILE * 37 + r);
+#pragma unroll
+                for (int c = 0; c < 4; ++c)
+                    x[h][c] = *reinterpret_cast<const longlong2*>(st + Q1T_TILE * 4 + c * Q1T_TILE * 8 + r * 8);
+            }
+            mbar_arrive(&empty[s]);  // this thread's reads of the stage are in registers
+#pragma unroll
+            for (int h = 0; h < 2; ++h) {
+                const int key0 = (int)(kk1[h] & 0xFF) * a.m1 + (int)(kk2[h] & 0xFF) * a.m2 + a.koff;
+                const int key1 = (int)(kk1[h] >> 8) * a.m1 + (int)(kk2[h] >> 8) * a.m2 + a.koff;
+                q1_row_smem<NARROW>(acc_t, a, G, dd[h].x, key0, x[h][0].x, x[h][1].x, x[h][2].x, x[h][3].x);
+                q1_row_smem<NARROW>(acc_t, a, G, dd[h].y, key1, x[h][0].y, x[h][1].y, x[h][2].y, x[h][3].y);
+            }
+        }
+        // ragged tail: rows past the last full tile, CTA 0 only
+        if (blockIdx.x == 0) {
+            for (int64_t r = ntiles * Q1T_TILE + threadIdx.x; r < a.n; r += Q1T_NT) {
+                const int key = (int)a.k1[r] * a.m1 + (int)a.k2[r] * a.m2 + a.koff;
+                q1_row_smem<NARROW>(acc_t, a, G, a.d[r], key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
+            }
+        }
+    }
+    __syncthreads();
+
+    // ---- hierarchical fold: thread slots -> warp (int64, proven) -> CTA (i128) -> grid ----
+    __shared__ i128 s_part[Q1T_CW][G][6];
+    if (warp < Q1T_CW) {
+#pragma unroll
+        for (int g = 0; g < G; ++g) {
+            const int64_t* p = acc + (size_t)g * Q1T_WORDS * Q1T_NT + threadIdx.x;
+            const int64_t dcw = p[4 * Q1T_NT];
+            int64_t v[6] = {p[0], p[Q1T_NT], p[2 * Q1T_NT], p[3 * Q1T_NT], dcw & ((1ll << Q1_CSHIFT) - 1),
+                            dcw >> Q1_CSHIFT};
+#pragma unroll
+            for (int k = 0; k < 6; ++k) {
+                int64_t w = warp_sum_i64(v[k]);
+                if (lane == 0) s_part[warp][g][k] = (i128)w;
+            }
+        }
+    }
+    __syncthreads();
+    if (threadIdx.x < G * 6) {
+        const int g = threadIdx.x / 6, k = threadIdx.x % 6;
+        i128 t = 0;
+        for (int w = 0; w < Q1T_CW; ++w) t += s_part[w][g][k];
+        put_i128(&parts[(size_t)blockIdx.x * G * 6 + threadIdx.x], t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < G * 6) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[threadIdx.x], t);
+    }
+}
+
 // Map the Q1 fragment's raw [G][6] sums to the plan's [ngroups][naggs+1].
 struct Q1Map {
     int32_t naggs, ngroups;
@@ -685,6 +859,162 @@ __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constan
             else put_i128(&r, get_i128(r) + get_i128(x));
         }
         out[threadIdx.x] = r;  // raw [sum, count], remapped by k_scalar_remap
+    }
+}
+
+// ---- scalar fragment, TMA-staged -------------------------------------------------
+// Up to 5 distinct columns (the filter columns and the value columns, shared
+// when a value column is also a filter column, as l_discount in Q6) streamed
+// through an SC_STAGES-deep ring of SC_TILE-row slices by one producer warp;
+// consumer thread t folds rows t, t+NT, ... of each staged tile.
+constexpr int SCT_CW = 8;
+constexpr int SCT_NT = SCT_CW * 32;
+constexpr int SCT_THREADS = SCT_NT + 32;
+constexpr int SCT_TILE = 2048;
+constexpr int SCT_MAXSTAGES = 16;
+
+struct ScalarTmaArgs {
+    const void* col[5];   // distinct staged columns
+    int32_t esz[5];       // element sizes
+    int32_t soff[5];      // slice offsets within a stage (bytes)
+    int32_t ncol;
+    int32_t stage_bytes;
+    int32_t nstages;      // ring depth (~180 KB of tiles in flight per SM)
+    int32_t role[5];      // staged column of f0, f1, f2, va, vb
+    int64_t lo[3], hi[3];
+    int32_t fcmp[2];
+    double fc[2];
+    int64_t n;
+};
+
+template <typename T>
+__device__ __forceinline__ T role_ld(const uint8_t* st, const ScalarTmaArgs& a, int role, int r) {
+    return reinterpret_cast<const T*>(st + a.soff[a.role[role]])[r];
+}
+template <typename T>
+__device__ __forceinline__ T role_ldg(const ScalarTmaArgs& a, int role, int64_t r) {
+    return reinterpret_cast<const T*>(a.col[a.role[role]])[r];
+}
+
+template <int MODE, int NF, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+__global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid_constant__ ScalarTmaArgs a,
+                                                                    int64_t ntiles, Slot16* __restrict__ parts,
+                                                                    unsigned int* __restrict__ done,
+                                                                    Slot16* __restrict__ out) {
+    typedef typename AccOf<VA>::type ACC;
+    extern __shared__ __align__(128) uint8_t smem[];
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * a.stage_bytes);
+    uint64_t* empty = full + a.nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < a.nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], SCT_NT);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    ACC sum = 0;
+    int64_t cnt = 0;
+    auto row = [&](F0 x0, F1 x1, F2 x2, VA va, VB vb) {
+        bool p = ftest(x0, 0, a.lo, a.hi, a.fcmp, a.fc);
+        if (NF > 1) p = p && ftest(x1, 1, a.lo, a.hi, a.fcmp, a.fc);
+        if (NF > 2) p = p && ftest(x2, 2, a.lo, a.hi, a.fcmp, a.fc);
+        ACC v = (ACC)va;
+        if (HVB) v *= (ACC)vb;
+        if (MODE == 1) {  // predicated: contribution x predicate
+            sum += p ? v : (ACC)0;
+            cnt += p;
+        } else if (p) {   // branching
+            sum += v;
+            cnt += 1;
+        }
+    };
+    if (warp == SCT_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % a.nstages);
+                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * a.stage_bytes;
+                mbar_expect_tx(&full[s], (uint32_t)a.stage_bytes);
+                for (int c = 0; c < a.ncol; ++c)
+                    tma_load_1d(st + a.soff[c], (const uint8_t*)a.col[c] + tile * SCT_TILE * a.esz[c],
+                                (uint32_t)(SCT_TILE * a.esz[c]), &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % a.nstages);
+            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            const uint8_t* st = smem + (size_t)s * a.stage_bytes;
+            constexpr int RPT = SCT_TILE / SCT_NT;
+            F0 x0[RPT]; F1 x1[RPT]; F2 x2[RPT]; VA va[RPT]; VB vb[RPT];
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) {
+                const int r = threadIdx.x + k * SCT_NT;
+                x0[k] = role_ld<F0>(st, a, 0, r);
+                x1[k] = NF > 1 ? role_ld<F1>(st, a, 1, r) : F1(0);
+                x2[k] = NF > 2 ? role_ld<F2>(st, a, 2, r) : F2(0);
+                va[k] = role_ld<VA>(st, a, 3, r);
+                vb[k] = HVB ? role_ld<VB>(st, a, 4, r) : VB(1);
+            }
+            mbar_arrive(&empty[s]);
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) row(x0[k], x1[k], x2[k], va[k], vb[k]);
+        }
+        if (blockIdx.x == 0) {
+            for (int64_t r = ntiles * SCT_TILE + threadIdx.x; r < a.n; r += SCT_NT)
+                row(role_ldg<F0>(a, 0, r), NF > 1 ? role_ldg<F1>(a, 1, r) : F1(0),
+                    NF > 2 ? role_ldg<F2>(a, 2, r) : F2(0), role_ldg<VA>(a, 3, r), HVB ? role_ldg<VB>(a, 4, r) : VB(1));
+        }
+    }
+    // warp -> CTA -> grid
+    __shared__ Slot16 s_w[SCT_THREADS / 32][2];
+    int64_t c = warp_sum_i64(cnt);
+    if (IsFloat<VA>::value) {
+        double sm = warp_sum_f64((double)sum);
+        if (lane == 0) put_f64(&s_w[warp][0], sm);
+    } else {
+        i128 sm = warp_sum_i128((i128)(int64_t)sum);
+        if (lane == 0) put_i128(&s_w[warp][0], sm);
+    }
+    if (lane == 0) put_i128(&s_w[warp][1], (i128)c);
+    __syncthreads();
+    if (threadIdx.x < 2) {
+        Slot16 r = s_w[0][threadIdx.x];
+        for (int w = 1; w < SCT_THREADS / 32; ++w) {
+            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(s_w[w][0]));
+            else put_i128(&r, get_i128(r) + get_i128(s_w[w][threadIdx.x]));
+        }
+        parts[(size_t)blockIdx.x * 2 + threadIdx.x] = r;
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < 2) {
+        Slot16 r;
+        r.lo = __ldcg(&parts[threadIdx.x].lo);
+        r.hi = __ldcg(&parts[threadIdx.x].hi);
+        for (unsigned b = 1; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
+            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
+            else put_i128(&r, get_i128(r) + get_i128(x));
+        }
+        out[threadIdx.x] = r;
     }
 }
 
@@ -885,9 +1215,26 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
     Slot16* raw = parts + (size_t)grid * G * 6;
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-#define Q1_LAUNCH(GG)                                                                                    \
-    if (narrow) k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                     \
-    else k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                           \
+    const char* var = getenv("VD_Q1_VARIANT");
+    // 1D bulk copies need 16-byte aligned sources: every column, including the u8 keys
+    const bool al_all = al(cols[p->key[0].col].data, 16) && al(cols[p->key[1].col].data, 16);
+    const bool use_tma = al_all && !(var && strcmp(var, "ldg") == 0);
+    const int64_t ntiles = n / Q1T_TILE;
+    const int tgrid = num_sms();
+#define Q1_LAUNCH(GG)                                                                                          \
+    if (use_tma) {                                                                                             \
+        if (narrow) {                                                                                          \
+            cudaFuncSetAttribute(k_pipe_q1_tma<GG, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
+            k_pipe_q1_tma<GG, true><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, raw);           \
+        } else {                                                                                               \
+            cudaFuncSetAttribute(k_pipe_q1_tma<GG, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
+            k_pipe_q1_tma<GG, false><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, raw);          \
+        }                                                                                                      \
+    } else if (narrow) {                                                                                       \
+        k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                                   \
+    } else {                                                                                                   \
+        k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                                  \
+    }                                                                                                          \
     k_q1_remap<GG><<<1, 1024, 0, s>>>(raw, map, (Slot16*)out);
     if (G == 4) { Q1_LAUNCH(4) } else if (G == 6) { Q1_LAUNCH(6) } else { Q1_LAUNCH(8) }
 #undef Q1_LAUNCH
@@ -899,6 +1246,50 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
 }
 
 // ---- scalar matching ----------------------------------------------------------
+// Stage layout for the TMA scalar fragment: distinct columns of the 5 roles.
+static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5], bool present[5], ScalarTmaArgs* t) {
+    t->ncol = 0;
+    int off = 0;
+    for (int r = 0; r < 5; ++r) {
+        t->role[r] = 0;
+        if (!present[r]) continue;
+        int found = -1;
+        for (int c = 0; c < t->ncol; ++c)
+            if (t->col[c] == role_ptr[r]) found = c;
+        if (found < 0) {
+            if (((uintptr_t)role_ptr[r] % 16) != 0) return false;
+            found = t->ncol++;
+            t->col[found] = role_ptr[r];
+            t->esz[found] = role_esz[r];
+            t->soff[found] = off;
+            off += SCT_TILE * role_esz[r];
+        }
+        t->role[r] = found;
+    }
+    t->stage_bytes = off;
+    int ns = (int)((180 * 1024) / (off > 0 ? off : 1));
+    t->nstages = ns < 2 ? 2 : (ns > SCT_MAXSTAGES ? SCT_MAXSTAGES : ns);
+    return (size_t)off * t->nstages + 2 * t->nstages * 8 <= 220 * 1024;
+}
+
+template <int MODE, int NF, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* out, const ScalarMap& m,
+                                     cudaStream_t s, int* nl) {
+    int grid = num_sms();
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    Slot16* raw = parts + (size_t)grid * 2;
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) return e;
+    size_t smem = (size_t)ta.stage_bytes * ta.nstages + 2 * ta.nstages * 8;
+    auto kern = k_pipe_scalar_tma<MODE, NF, HVB, F0, F1, F2, VA, VB>;
+    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    kern<<<grid, SCT_THREADS, smem, s>>>(ta, ta.n / SCT_TILE, parts, dn, raw);
+    k_scalar_remap<<<1, 32, 0, s>>>(raw, m, out);
+    *nl += 2;
+    return cudaGetLastError();
+}
+
 template <int MODE, bool HF1, bool HF2, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
 static cudaError_t launch_scalar(const ScalarArgs<F0, F1, F2, VA, VB>& sa, void* ws, Slot16* out, const ScalarMap& m,
                                  cudaStream_t s, int* nl) {
@@ -978,6 +1369,8 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
     }
     cudaError_t e = cudaSuccess;
     Slot16* o = (Slot16*)out;
+    const char* var = getenv("VD_SCALAR_VARIANT");
+    const bool use_tma = !(var && strcmp(var, "ldg") == 0);
     // Q6 shape: filters (i32, i64, i64), value i64 * i64
     if (nf == 3 && t0 == VD_I32 && t1 == VD_I64 && t2 == VD_I64 && tva == VD_I64 && tvb == VD_I64 &&
         al16(cols[fcol[0]].data)) {
@@ -991,7 +1384,18 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
         sa.va = (const int64_t*)cols[va].data;
         sa.vb = (const int64_t*)cols[vb].data;
         sa.n = n;
-        if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
+        ScalarTmaArgs ta;
+        const void* rp[5] = {sa.f0, sa.f1, sa.f2, sa.va, sa.vb};
+        const int re[5] = {4, 8, 8, 8, 8};
+        bool pr[5] = {true, true, true, true, true};
+        if (use_tma && scalar_tma_args(rp, re, pr, &ta)) {
+            for (int j = 0; j < 3; ++j) { ta.lo[j] = lo[j]; ta.hi[j] = hi[j]; }
+            ta.fcmp[0] = ta.fcmp[1] = -1;
+            ta.fc[0] = ta.fc[1] = 0;
+            ta.n = n;
+            if (mode) e = launch_scalar_tma<1, 3, true, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
+            else e = launch_scalar_tma<0, 3, true, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
+        } else if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
         else e = launch_scalar<0, true, true, true>(sa, ws, o, m, s, nl);
     } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && al16(cols[fcol[0]].data)) {
         // selective aggregation over one f32 column (Fig 15 / C1)
@@ -1004,7 +1408,18 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
         sa.va = (const float*)cols[va].data;
         sa.vb = nullptr;
         sa.n = n;
-        if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
+        ScalarTmaArgs ta;
+        const void* rp[5] = {sa.f0, nullptr, nullptr, sa.va, nullptr};
+        const int re[5] = {4, 4, 4, 4, 4};
+        bool pr[5] = {true, false, false, true, false};
+        if (use_tma && scalar_tma_args(rp, re, pr, &ta)) {
+            for (int j = 0; j < 3; ++j) { ta.lo[j] = lo[j]; ta.hi[j] = hi[j]; }
+            ta.fcmp[0] = fcmp[0]; ta.fcmp[1] = fcmp[1];
+            ta.fc[0] = fc[0]; ta.fc[1] = fc[1];
+            ta.n = n;
+            if (mode) e = launch_scalar_tma<1, 1, false, float, float, float, float, float>(ta, ws, o, m, s, nl);
+            else e = launch_scalar_tma<0, 1, false, float, float, float, float, float>(ta, ws, o, m, s, nl);
+        } else if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
         else e = launch_scalar<0, false, false, false>(sa, ws, o, m, s, nl);
     } else {
         return VD_OK;

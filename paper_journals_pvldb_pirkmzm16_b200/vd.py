@@ -207,6 +207,7 @@ def column(t, minmax: Optional[Sequence[int]] = None, scale: int = 0, length: Op
     if minmax is not None:
         c.min, c.max = int(minmax[0]), int(minmax[1])
         c.has_minmax = 1
+    c._keep = t  # the view keeps its tensor alive (the ABI struct holds a raw pointer)
     return c
 
 
@@ -217,6 +218,7 @@ def ctrl(from_: int = 0, num: int = 1, den: int = 1, cap: int = 0, materialized=
     if materialized is not None:
         c.materialized = materialized.data_ptr()
         c.mat_dtype = dtype_of(materialized)
+        c._keep = materialized
     return c
 
 
