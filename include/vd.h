@@ -361,6 +361,10 @@ vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int3
  * vd_pipeline.  Returns the number written (<= n). */
 int32_t vd_abi_struct_sizes(size_t* out, int32_t n);
 
+/* Name of the fragment the last vd_run_pipeline on this thread ran:
+ * "q1_tma", "q1_ldg", "scalar_tma", "scalar_ldg", "selsum_tma", "gather_fold" or "generic". */
+const char* vd_last_fragment(void);
+
 /* Number of kernel launches the last successful call on this thread
  * enqueued (for launch accounting in benchmarks). */
 int32_t vd_last_launch_count(void);

@@ -53,6 +53,15 @@ __device__ __forceinline__ void put_f64(Slot16* s, double v) {
 }
 __device__ __forceinline__ double get_f64(const Slot16& s) { return __longlong_as_double((long long)s.lo); }
 
+// Maps from a fragment's raw result slots to the plan's [ngroups][naggs+1].
+struct Q1Map {
+    int32_t naggs, ngroups;
+    int32_t src[VD_MAX_AGGS];  // raw slot (0..5) per plan aggregate
+};
+struct ScalarMap {
+    int32_t naggs;
+    int32_t src[VD_MAX_AGGS];  // 0 = sum, 1 = count
+};
 // ============================================================================
 // Generic fragment
 // ============================================================================
@@ -405,7 +414,8 @@ __device__ __forceinline__ void q1_row(Q1Acc<G, NARROW>& A, const Q1Args& a, boo
 
 template <int G, bool NARROW>
 __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant__ Q1Args a, Slot16* __restrict__ parts,
-                                                           unsigned int* __restrict__ done, Slot16* __restrict__ out) {
+                                                           unsigned int* __restrict__ done, Slot16* __restrict__ out,
+                                                           const Q1Map map) {
     Q1Acc<G, NARROW> A;
 #pragma unroll
     for (int g = 0; g < G; ++g) { A.s0[g] = A.s1[g] = A.s2[g] = A.s3[g] = A.dc[g] = 0; }
@@ -505,6 +515,7 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
     __syncthreads();
     if (!s_last) return;
     __threadfence();
+    __shared__ Slot16 s_raw[G * 6];
     if (threadIdx.x < G * 6) {
         i128 t = 0;
         for (unsigned b = 0; b < gridDim.x; ++b) {
@@ -513,7 +524,13 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
             x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
             t += get_i128(x);
         }
-        put_i128(&out[threadIdx.x], t);  // [G][6] raw slots, remapped by k_q1_remap
+        put_i128(&s_raw[threadIdx.x], t);
+    }
+    __syncthreads();
+    // the plan's [ngroups][naggs+1] layout (slot naggs = row count = COUNT)
+    for (int k = threadIdx.x; k < map.ngroups * (map.naggs + 1); k += blockDim.x) {
+        const int g = k / (map.naggs + 1), ag = k % (map.naggs + 1);
+        out[k] = s_raw[g * 6 + ((ag == map.naggs) ? 5 : map.src[ag])];
     }
 }
 
@@ -567,7 +584,7 @@ template <int G, bool NARROW>
 __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_constant__ Q1Args a, int64_t ntiles,
                                                                 Slot16* __restrict__ parts,
                                                                 unsigned int* __restrict__ done,
-                                                                Slot16* __restrict__ out) {
+                                                                Slot16* __restrict__ out, const Q1Map map) {
     extern __shared__ __align__(128) uint8_t smem[];
     int64_t* acc = reinterpret_cast<int64_t*>(smem + (size_t)Q1T_STAGES * Q1T_STAGE_BYTES);
     uint64_t* full = reinterpret_cast<uint64_t*>(acc + (size_t)(G + 1) * Q1T_WORDS * Q1T_NT);
@@ -576,7 +593,7 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
     if (threadIdx.x == 0) {
         for (int s = 0; s < Q1T_STAGES; ++s) {
             mbar_init(&full[s], 1);
-            mbar_init(&empty[s], Q1T_NT);
+            mbar_init(&empty[s], Q1T_CW);
         }
         fence_mbar_init();
     }
@@ -627,7 +644,8 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
                 for (int c = 0; c < 4; ++c)
                     x[h][c] = *reinterpret_cast<const longlong2*>(st + Q1T_TILE * 4 + c * Q1T_TILE * 8 + r * 8);
             }
-            mbar_arrive(&empty[s]);  // this thread's reads of the stage are in registers
+            __syncwarp();  // the warp's reads of the stage are done
+            if (lane == 0) mbar_arrive(&empty[s]);
 #pragma unroll
             for (int h = 0; h < 2; ++h) {
                 const int key0 = (int)(kk1[h] & 0xFF) * a.m1 + (int)(kk2[h] & 0xFF) * a.m2 + a.koff;
@@ -678,6 +696,7 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
     __syncthreads();
     if (!s_last) return;
     __threadfence();
+    __shared__ Slot16 s_raw[G * 6];
     if (threadIdx.x < G * 6) {
         i128 t = 0;
         for (unsigned b = 0; b < gridDim.x; ++b) {
@@ -686,24 +705,17 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
             x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
             t += get_i128(x);
         }
-        put_i128(&out[threadIdx.x], t);
+        put_i128(&s_raw[threadIdx.x], t);
+    }
+    __syncthreads();
+    // the plan's [ngroups][naggs+1] layout (slot naggs = row count = COUNT)
+    for (int k = threadIdx.x; k < map.ngroups * (map.naggs + 1); k += blockDim.x) {
+        const int g = k / (map.naggs + 1), ag = k % (map.naggs + 1);
+        out[k] = s_raw[g * 6 + ((ag == map.naggs) ? 5 : map.src[ag])];
     }
 }
 
 // Map the Q1 fragment's raw [G][6] sums to the plan's [ngroups][naggs+1].
-struct Q1Map {
-    int32_t naggs, ngroups;
-    int32_t src[VD_MAX_AGGS];  // raw slot (0..5) per plan aggregate
-};
-template <int G>
-__global__ void k_q1_remap(const Slot16* __restrict__ raw, Q1Map m, Slot16* __restrict__ out) {
-    int k = threadIdx.x;
-    int slots = m.ngroups * (m.naggs + 1);
-    if (k >= slots) return;
-    int g = k / (m.naggs + 1), a = k % (m.naggs + 1);
-    int s = (a == m.naggs) ? 5 : m.src[a];
-    out[k] = raw[g * 6 + s];
-}
 
 // ============================================================================
 // Scalar fragment (Q6 / selective aggregation):
@@ -747,8 +759,9 @@ template <int MODE, bool HAS_F1, bool HAS_F2, bool HAS_VB, typename F0, typename
           typename VB>
 __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constant__ ScalarArgs<F0, F1, F2, VA, VB> a,
                                                             Slot16* __restrict__ parts, unsigned int* __restrict__ done,
-                                                            Slot16* __restrict__ out) {
+                                                            Slot16* __restrict__ out, const ScalarMap map) {
     typedef typename AccOf<VA>::type ACC;
+    __shared__ Slot16 s_raw2[2];
     ACC sum = 0;
     int64_t cnt = 0;
     const int64_t nthreads = (int64_t)gridDim.x * SC_THREADS;
@@ -858,8 +871,10 @@ __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constan
             if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
             else put_i128(&r, get_i128(r) + get_i128(x));
         }
-        out[threadIdx.x] = r;  // raw [sum, count], remapped by k_scalar_remap
+        s_raw2[threadIdx.x] = r;
     }
+    __syncthreads();
+    if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
 }
 
 // ---- scalar fragment, TMA-staged -------------------------------------------------
@@ -896,12 +911,13 @@ __device__ __forceinline__ T role_ldg(const ScalarTmaArgs& a, int role, int64_t 
     return reinterpret_cast<const T*>(a.col[a.role[role]])[r];
 }
 
-template <int MODE, int NF, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+template <int MODE, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA, typename VB>
 __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid_constant__ ScalarTmaArgs a,
                                                                     int64_t ntiles, Slot16* __restrict__ parts,
                                                                     unsigned int* __restrict__ done,
-                                                                    Slot16* __restrict__ out) {
+                                                                    Slot16* __restrict__ out, const ScalarMap map) {
     typedef typename AccOf<VA>::type ACC;
+    __shared__ Slot16 s_raw2[2];
     extern __shared__ __align__(128) uint8_t smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * a.stage_bytes);
     uint64_t* empty = full + a.nstages;
@@ -909,7 +925,7 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
     if (threadIdx.x == 0) {
         for (int s = 0; s < a.nstages; ++s) {
             mbar_init(&full[s], 1);
-            mbar_init(&empty[s], SCT_NT);
+            mbar_init(&empty[s], SCT_CW);
         }
         fence_mbar_init();
     }
@@ -941,8 +957,8 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
                 uint8_t* st = smem + (size_t)s * a.stage_bytes;
                 mbar_expect_tx(&full[s], (uint32_t)a.stage_bytes);
                 for (int c = 0; c < a.ncol; ++c)
-                    tma_load_1d(st + a.soff[c], (const uint8_t*)a.col[c] + tile * SCT_TILE * a.esz[c],
-                                (uint32_t)(SCT_TILE * a.esz[c]), &full[s], pol);
+                    tma_load_1d(st + a.soff[c], (const uint8_t*)a.col[c] + tile * TILE * a.esz[c],
+                                (uint32_t)(TILE * a.esz[c]), &full[s], pol);
             }
         }
         __syncwarp();
@@ -953,7 +969,7 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
             const int s = (int)(it % a.nstages);
             mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
             const uint8_t* st = smem + (size_t)s * a.stage_bytes;
-            constexpr int RPT = SCT_TILE / SCT_NT;
+            constexpr int RPT = TILE / SCT_NT;
             F0 x0[RPT]; F1 x1[RPT]; F2 x2[RPT]; VA va[RPT]; VB vb[RPT];
 #pragma unroll
             for (int k = 0; k < RPT; ++k) {
@@ -964,12 +980,13 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
                 va[k] = role_ld<VA>(st, a, 3, r);
                 vb[k] = HVB ? role_ld<VB>(st, a, 4, r) : VB(1);
             }
-            mbar_arrive(&empty[s]);
+            __syncwarp();  // the warp's reads of the stage are done
+            if (lane == 0) mbar_arrive(&empty[s]);
 #pragma unroll
             for (int k = 0; k < RPT; ++k) row(x0[k], x1[k], x2[k], va[k], vb[k]);
         }
         if (blockIdx.x == 0) {
-            for (int64_t r = ntiles * SCT_TILE + threadIdx.x; r < a.n; r += SCT_NT)
+            for (int64_t r = ntiles * TILE + threadIdx.x; r < a.n; r += SCT_NT)
                 row(role_ldg<F0>(a, 0, r), NF > 1 ? role_ldg<F1>(a, 1, r) : F1(0),
                     NF > 2 ? role_ldg<F2>(a, 2, r) : F2(0), role_ldg<VA>(a, 3, r), HVB ? role_ldg<VB>(a, 4, r) : VB(1));
         }
@@ -1014,18 +1031,266 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
             if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
             else put_i128(&r, get_i128(r) + get_i128(x));
         }
-        out[threadIdx.x] = r;
+        s_raw2[threadIdx.x] = r;
     }
+    __syncthreads();
+    if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
 }
 
-struct ScalarMap {
+
+// ============================================================================
+// Gather-fold fragment (FK joins: Q19 / Q9 style, a4 + a7 fused)
+// ============================================================================
+// Base columns are streamed through a TMA ring (as the scalar fragment);
+// per row the predicate's base-column terms are evaluated before any gather
+// (late materialisation: the random accesses into the dimension tables --
+// identity-hashed FK positions, P:L1054-1056 -- happen only for rows that
+// can still qualify), then the gathered terms, the group key (identity or
+// calendar year, the latter through a shared-memory lookup table), and
+// int64 products (exactness proven from min/max metadata on the host).
+// Groups are folded per warp: lanes with equal keys are matched
+// (__match_any_sync) and one leader per key adds their staged values into
+// the warp's shared-memory slots -- no atomics.
+constexpr int GF_CW = 8;
+constexpr int GF_NT = GF_CW * 32;
+constexpr int GF_THREADS = GF_NT + 32;
+constexpr int GF_TILE = 2048;
+constexpr int GF_MAXSTAGES = 8;
+constexpr int GF_MAXCOLS = 8;
+constexpr int GF_MAXYEARDAYS = 8192;
+
+struct GfArgs {
+    // staged base columns
+    const void* col[GF_MAXCOLS];
+    int32_t dt[GF_MAXCOLS], esz[GF_MAXCOLS], soff[GF_MAXCOLS];
+    int32_t ncols;
+    int32_t stage_bytes, nstages;
+    // gathers: reference c = ncols + g
+    int32_t ngathers;
+    int32_t g_fk[VD_MAX_GATHERS];
+    int64_t g_bias[VD_MAX_GATHERS];
+    const void* g_p[VD_MAX_GATHERS];
+    int64_t g_len[VD_MAX_GATHERS];
+    int32_t g_dt[VD_MAX_GATHERS];
+    // predicate: per conjunction, base terms first (nbase[c] of them)
+    DevPred pred;
+    int32_t nbase[VD_MAX_CONJ];
+    // key
+    int32_t nkey;
+    int32_t k_col[VD_MAX_KEYPARTS], k_fn[VD_MAX_KEYPARTS];
+    int64_t k_sub[VD_MAX_KEYPARTS], k_mult[VD_MAX_KEYPARTS];
+    int32_t year_lo, year_days;  // calendar table covers [year_lo, year_lo + year_days)
+    int32_t ngroups;
+    // aggregates: SUM of prod (a + b*col) (int64), or COUNT
     int32_t naggs;
-    int32_t src[VD_MAX_AGGS];  // 0 = sum, 1 = count
+    int32_t a_kind[VD_MAX_AGGS], a_nf[VD_MAX_AGGS];
+    int32_t a_col[VD_MAX_AGGS][VD_MAX_FACTORS];
+    int64_t a_a[VD_MAX_AGGS][VD_MAX_FACTORS], a_b[VD_MAX_AGGS][VD_MAX_FACTORS];
+    int64_t n;
 };
-__global__ void k_scalar_remap(const Slot16* __restrict__ raw, ScalarMap m, Slot16* __restrict__ out) {
-    int k = threadIdx.x;
-    if (k > m.naggs) return;
-    out[k] = raw[(k == m.naggs) ? 1 : m.src[k]];
+
+struct GfRow {
+    const uint8_t* st;  // stage base (nullptr: read global, tail rows)
+    int r;              // row within the tile
+    int64_t g;          // global row
+};
+
+__device__ __forceinline__ Val gf_base(const GfArgs& a, const GfRow& w, int c) {
+    if (w.st) {
+        const uint8_t* q = w.st + a.soff[c];
+        Val v;
+        v.isf = false;
+        v.f = 0;
+        switch (a.dt[c]) {
+        case VD_U8: { uint8_t x = q[w.r]; v.eps = x == 0xFF; v.i = x; break; }
+        case VD_I32: { int32_t x = reinterpret_cast<const int32_t*>(q)[w.r]; v.eps = x == INT32_MIN; v.i = x; break; }
+        case VD_I64: { int64_t x = reinterpret_cast<const int64_t*>(q)[w.r]; v.eps = x == INT64_MIN; v.i = x; break; }
+        case VD_F32: { float x = reinterpret_cast<const float*>(q)[w.r]; v.eps = x != x; v.isf = true; v.f = x; v.i = 0; break; }
+        default: { double x = reinterpret_cast<const double*>(q)[w.r]; v.eps = x != x; v.isf = true; v.f = x; v.i = 0; break; }
+        }
+        return v;
+    }
+    return fetch_typed(a.col[c], a.dt[c], w.g);
+}
+
+__device__ __forceinline__ Val gf_fetch(const GfArgs& a, const GfRow& w, int c) {
+    if (c < a.ncols) return gf_base(a, w, c);
+    const int g = c - a.ncols;
+    Val fk = gf_base(a, w, a.g_fk[g]);
+    Val out;
+    out.eps = true;
+    out.isf = false;
+    out.i = 0;
+    out.f = 0;
+    if (fk.eps) return out;
+    const int64_t p = fk.i - a.g_bias[g];
+    if (p < 0 || p >= a.g_len[g]) return out;
+    return fetch_typed(a.g_p[g], a.g_dt[g], p);
+}
+
+__device__ __forceinline__ bool gf_pred(const GfArgs& a, const GfRow& w) {
+    if (a.pred.nconj == 0) return true;
+    // phase 1: base-column terms of every conjunction (no gathers)
+    unsigned alive = 0;
+    for (int c = 0; c < a.pred.nconj; ++c) {
+        bool ok = true;
+        for (int k = 0; k < a.nbase[c] && ok; ++k) ok = term_true(a.pred.t[c][k], gf_base(a, w, a.pred.t[c][k].col));
+        if (ok) {
+            if (a.nbase[c] == a.pred.nterms[c]) return true;
+            alive |= 1u << c;
+        }
+    }
+    // phase 2: gathered terms, only for conjunctions still alive
+    for (int c = 0; c < a.pred.nconj; ++c) {
+        if (!((alive >> c) & 1u)) continue;
+        bool ok = true;
+        for (int k = a.nbase[c]; k < a.pred.nterms[c] && ok; ++k) {
+            const DevTerm& t = a.pred.t[c][k];
+            ok = term_true(t, gf_fetch(a, w, t.col));
+        }
+        if (ok) return true;
+    }
+    return false;
+}
+
+template <int MODE>
+__global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant__ GfArgs a, int64_t ntiles,
+                                                           Slot16* __restrict__ parts, unsigned int* __restrict__ done,
+                                                           Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    const int NA = a.naggs, NS = a.ngroups * (a.naggs + 1);
+    int64_t* acc = reinterpret_cast<int64_t*>(smem + (size_t)a.nstages * a.stage_bytes);  // [GF_CW][NS]
+    int64_t* stage_v = acc + (size_t)GF_CW * NS;                                           // [GF_CW][32][NA+1]
+    int16_t* ytab = reinterpret_cast<int16_t*>(stage_v + (size_t)GF_CW * 32 * (NA + 1));  // calendar years
+    uint64_t* full = reinterpret_cast<uint64_t*>(ytab + ((a.year_days + 7) & ~7));
+    uint64_t* empty = full + a.nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < a.nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], GF_CW);
+        }
+        fence_mbar_init();
+    }
+    for (int k = threadIdx.x; k < GF_CW * NS; k += GF_THREADS) acc[k] = 0;
+    for (int k = threadIdx.x; k < a.year_days; k += GF_THREADS) ytab[k] = (int16_t)year_of_day(a.year_lo + k);
+    __syncthreads();
+
+    auto process = [&](const GfRow& w, bool valid) {
+        bool ok = valid && gf_pred(a, w);
+        int64_t key = 0;
+        if (ok) {
+            for (int k = 0; k < a.nkey && ok; ++k) {
+                Val v = gf_fetch(a, w, a.k_col[k]);
+                if (v.eps) { ok = false; break; }
+                int64_t x = v.i;
+                if (a.k_fn[k] == 1) {
+                    const int64_t d = x - a.year_lo;
+                    x = (d >= 0 && d < a.year_days) ? (int64_t)ytab[d] : (int64_t)year_of_day((int32_t)x);
+                }
+                key += (x - a.k_sub[k]) * a.k_mult[k];
+            }
+            if (ok && (key < 0 || key >= a.ngroups)) ok = false;  // excluded by the host's domain proof
+        }
+        int64_t* sv = stage_v + ((size_t)warp * 32 + lane) * (NA + 1);
+        if (ok) {
+            for (int g = 0; g < NA; ++g) {
+                int64_t pr = 1;
+                if (a.a_kind[g] != VD_AGG_COUNT) {
+                    for (int f = 0; f < a.a_nf[g]; ++f) {
+                        int64_t x = 0;
+                        if (a.a_col[g][f] >= 0) x = gf_fetch(a, w, a.a_col[g][f]).i;
+                        pr *= a.a_a[g][f] + a.a_b[g][f] * x;
+                    }
+                }
+                sv[g] = pr;
+            }
+            sv[NA] = 1;
+        }
+        __syncwarp();
+        const unsigned m = __match_any_sync(VD_FULL, ok ? key : -1ll);
+        if (ok && (__ffs(m) - 1) == lane) {
+            int64_t* dst = acc + (size_t)warp * NS + key * (NA + 1);
+            for (int g = 0; g <= NA; ++g) {
+                int64_t t = 0;
+                for (unsigned mm = m; mm; mm &= mm - 1)
+                    t += stage_v[((size_t)warp * 32 + (__ffs(mm) - 1)) * (NA + 1) + g];
+                dst[g] += t;
+            }
+        }
+        __syncwarp();
+    };
+
+    if (warp == GF_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % a.nstages);
+                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * a.stage_bytes;
+                mbar_expect_tx(&full[s], (uint32_t)a.stage_bytes);
+                for (int c = 0; c < a.ncols; ++c)
+                    tma_load_1d(st + a.soff[c], (const uint8_t*)a.col[c] + tile * GF_TILE * a.esz[c],
+                                (uint32_t)(GF_TILE * a.esz[c]), &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % a.nstages);
+            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            const uint8_t* st = smem + (size_t)s * a.stage_bytes;
+            for (int k = 0; k < GF_TILE / GF_NT; ++k) {
+                GfRow w;
+                w.st = st;
+                w.r = threadIdx.x + k * GF_NT;
+                w.g = tile * GF_TILE + w.r;
+                process(w, true);
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+        }
+        if (blockIdx.x == 0) {
+            const int64_t t0 = ntiles * GF_TILE;
+            for (int64_t base = t0 + warp * 32; base < a.n; base += GF_NT) {  // warp-uniform trip count
+                GfRow w;
+                w.st = nullptr;
+                w.r = 0;
+                w.g = base + lane;
+                process(w, w.g < a.n);
+            }
+        }
+    }
+    __syncthreads();
+    // CTA fold of the warps' slots (int128), then the grid's (last CTA)
+    for (int k = threadIdx.x; k < NS; k += GF_THREADS) {
+        i128 t = 0;
+        for (int w = 0; w < GF_CW; ++w) t += (i128)acc[(size_t)w * NS + k];
+        put_i128(&parts[(size_t)blockIdx.x * NS + k], t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    for (int k = threadIdx.x; k < NS; k += GF_THREADS) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
+            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[k], t);
+    }
 }
 
 // ============================================================================
@@ -1225,20 +1490,21 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
     if (use_tma) {                                                                                             \
         if (narrow) {                                                                                          \
             cudaFuncSetAttribute(k_pipe_q1_tma<GG, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
-            k_pipe_q1_tma<GG, true><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, raw);           \
+            k_pipe_q1_tma<GG, true><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, (Slot16*)out, map);           \
         } else {                                                                                               \
             cudaFuncSetAttribute(k_pipe_q1_tma<GG, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
-            k_pipe_q1_tma<GG, false><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, raw);          \
+            k_pipe_q1_tma<GG, false><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, (Slot16*)out, map);          \
         }                                                                                                      \
     } else if (narrow) {                                                                                       \
-        k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                                   \
+        k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, (Slot16*)out, map);                                   \
     } else {                                                                                                   \
-        k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, raw);                                  \
-    }                                                                                                          \
-    k_q1_remap<GG><<<1, 1024, 0, s>>>(raw, map, (Slot16*)out);
+        k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, (Slot16*)out, map);                                  \
+    }
     if (G == 4) { Q1_LAUNCH(4) } else if (G == 6) { Q1_LAUNCH(6) } else { Q1_LAUNCH(8) }
+    set_fragment(use_tma ? "q1_tma" : "q1_ldg");
 #undef Q1_LAUNCH
-    *nl += 2;
+    *nl += 1;
+    (void)raw;
     e = cudaGetLastError();
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     *done = true;
@@ -1246,8 +1512,167 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
 }
 
 // ---- scalar matching ----------------------------------------------------------
+// ---- selective sum over one f32 column, TMA-staged (Fig 15 / C1) -------------
+// select v in [lo, hi] (inclusive f32 bounds; every single-term comparison on
+// an f32 value is such an interval: x > c <=> x >= succ(floor32(c))), fold
+// the selected values in f64 and count them.  4 rows per LDS.128.
+constexpr int SS_TILE = 8192;
+constexpr int SS_MAXSTAGES = 6;
+
+struct SelSumArgs {
+    const float* v;
+    float lo, hi;
+    int64_t n;
+    int32_t nstages;
+};
+
+template <int MODE>
+__global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid_constant__ SelSumArgs a,
+                                                                    int64_t ntiles, Slot16* __restrict__ parts,
+                                                                    unsigned int* __restrict__ done,
+                                                                    Slot16* __restrict__ out, const ScalarMap map) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    __shared__ Slot16 s_raw2[2];
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * SS_TILE * 4);
+    uint64_t* empty = full + a.nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < a.nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], SCT_CW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    double sum = 0;
+    int64_t cnt = 0;
+    auto row = [&](float x) {
+        const bool p = x >= a.lo && x <= a.hi;  // NaN (epsilon) fails both
+        if (MODE == 1) {
+            sum += p ? (double)x : 0.0;
+            cnt += p;
+        } else if (p) {
+            sum += (double)x;
+            cnt += 1;
+        }
+    };
+    if (warp == SCT_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % a.nstages);
+                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                mbar_expect_tx(&full[s], SS_TILE * 4);
+                tma_load_1d(smem + (size_t)s * SS_TILE * 4, a.v + tile * SS_TILE, SS_TILE * 4, &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % a.nstages);
+            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            const float4* st = reinterpret_cast<const float4*>(smem + (size_t)s * SS_TILE * 4);
+            float4 x[SS_TILE / 4 / SCT_NT];
+#pragma unroll
+            for (int k = 0; k < SS_TILE / 4 / SCT_NT; ++k) x[k] = st[threadIdx.x + k * SCT_NT];
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+#pragma unroll
+            for (int k = 0; k < SS_TILE / 4 / SCT_NT; ++k) {
+                row(x[k].x);
+                row(x[k].y);
+                row(x[k].z);
+                row(x[k].w);
+            }
+        }
+        if (blockIdx.x == 0)
+            for (int64_t r = ntiles * SS_TILE + threadIdx.x; r < a.n; r += SCT_NT) row(a.v[r]);
+    }
+    __shared__ Slot16 s_w[SCT_THREADS / 32][2];
+    const int64_t c = warp_sum_i64(cnt);
+    const double sm = warp_sum_f64(sum);
+    if (lane == 0) {
+        put_f64(&s_w[warp][0], sm);
+        put_i128(&s_w[warp][1], (i128)c);
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        double t = 0;
+        i128 k = 0;
+        for (int w = 0; w < SCT_THREADS / 32; ++w) { t += get_f64(s_w[w][0]); k += get_i128(s_w[w][1]); }
+        put_f64(&parts[(size_t)blockIdx.x * 2], t);
+        put_i128(&parts[(size_t)blockIdx.x * 2 + 1], k);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < 2) {
+        Slot16 r;
+        r.lo = __ldcg(&parts[threadIdx.x].lo);
+        r.hi = __ldcg(&parts[threadIdx.x].hi);
+        for (unsigned b = 1; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
+            if (threadIdx.x == 0) put_f64(&r, get_f64(r) + get_f64(x));
+            else put_i128(&r, get_i128(r) + get_i128(x));
+        }
+        s_raw2[threadIdx.x] = r;
+    }
+    __syncthreads();
+    if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
+}
+
+// Inclusive f32 interval [lo, hi] equal to <= 2 comparison terms on an f32
+// column: for f32 x and a double constant c, x > c <=> x >= succ(floor32(c)),
+// x >= c <=> x >= ceil32(c), x < c <=> x <= pred(ceil32(c)),
+// x <= c <=> x <= floor32(c).  NaN (epsilon) fails both comparisons.
+static float floor32(double c) {
+    float f = (float)c;
+    if ((double)f > c) f = nextafterf(f, -INFINITY);
+    return f;
+}
+static float ceil32(double c) {
+    float f = (float)c;
+    if ((double)f < c) f = nextafterf(f, INFINITY);
+    return f;
+}
+static bool f32_interval(const int32_t fcmp[2], const double fc[2], float* lo, float* hi) {
+    float l = -INFINITY, h = INFINITY;
+    for (int k = 0; k < 2; ++k) {
+        if (fcmp[k] < 0) continue;
+        const double c = fc[k];
+        switch (fcmp[k]) {
+        case VD_CMP_GT: l = fmaxf(l, nextafterf(floor32(c), INFINITY)); break;
+        case VD_CMP_GE: l = fmaxf(l, ceil32(c)); break;
+        case VD_CMP_LT: h = fminf(h, nextafterf(ceil32(c), -INFINITY)); break;
+        case VD_CMP_LE: h = fminf(h, floor32(c)); break;
+        case VD_CMP_EQ:
+            if ((double)(float)c != c) { l = 1; h = 0; break; }  // no f32 equals c
+            l = fmaxf(l, (float)c);
+            h = fminf(h, (float)c);
+            break;
+        default: return false;
+        }
+    }
+    *lo = l;
+    *hi = h;
+    return true;
+}
+
 // Stage layout for the TMA scalar fragment: distinct columns of the 5 roles.
-static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5], bool present[5], ScalarTmaArgs* t) {
+static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5], bool present[5], int tile,
+                            ScalarTmaArgs* t) {
     t->ncol = 0;
     int off = 0;
     for (int r = 0; r < 5; ++r) {
@@ -1262,7 +1687,7 @@ static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5]
             t->col[found] = role_ptr[r];
             t->esz[found] = role_esz[r];
             t->soff[found] = off;
-            off += SCT_TILE * role_esz[r];
+            off += tile * role_esz[r];
         }
         t->role[r] = found;
     }
@@ -1272,7 +1697,7 @@ static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5]
     return (size_t)off * t->nstages + 2 * t->nstages * 8 <= 220 * 1024;
 }
 
-template <int MODE, int NF, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+template <int MODE, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA, typename VB>
 static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* out, const ScalarMap& m,
                                      cudaStream_t s, int* nl) {
     int grid = num_sms();
@@ -1282,11 +1707,11 @@ static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* 
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) return e;
     size_t smem = (size_t)ta.stage_bytes * ta.nstages + 2 * ta.nstages * 8;
-    auto kern = k_pipe_scalar_tma<MODE, NF, HVB, F0, F1, F2, VA, VB>;
+    auto kern = k_pipe_scalar_tma<MODE, NF, HVB, TILE, F0, F1, F2, VA, VB>;
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    kern<<<grid, SCT_THREADS, smem, s>>>(ta, ta.n / SCT_TILE, parts, dn, raw);
-    k_scalar_remap<<<1, 32, 0, s>>>(raw, m, out);
-    *nl += 2;
+    kern<<<grid, SCT_THREADS, smem, s>>>(ta, ta.n / TILE, parts, dn, out, m);
+    (void)raw;
+    *nl += 1;
     return cudaGetLastError();
 }
 
@@ -1299,9 +1724,9 @@ static cudaError_t launch_scalar(const ScalarArgs<F0, F1, F2, VA, VB>& sa, void*
     Slot16* raw = parts + (size_t)grid * 2;
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) return e;
-    k_pipe_scalar<MODE, HF1, HF2, HVB, F0, F1, F2, VA, VB><<<grid, SC_THREADS, 0, s>>>(sa, parts, dn, raw);
-    k_scalar_remap<<<1, 32, 0, s>>>(raw, m, out);
-    *nl += 2;
+    k_pipe_scalar<MODE, HF1, HF2, HVB, F0, F1, F2, VA, VB><<<grid, SC_THREADS, 0, s>>>(sa, parts, dn, out, m);
+    (void)raw;
+    *nl += 1;
     return cudaGetLastError();
 }
 
@@ -1371,6 +1796,7 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
     Slot16* o = (Slot16*)out;
     const char* var = getenv("VD_SCALAR_VARIANT");
     const bool use_tma = !(var && strcmp(var, "ldg") == 0);
+    float sslo = 0, sshi = 0;
     // Q6 shape: filters (i32, i64, i64), value i64 * i64
     if (nf == 3 && t0 == VD_I32 && t1 == VD_I64 && t2 == VD_I64 && tva == VD_I64 && tvb == VD_I64 &&
         al16(cols[fcol[0]].data)) {
@@ -1388,15 +1814,44 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
         const void* rp[5] = {sa.f0, sa.f1, sa.f2, sa.va, sa.vb};
         const int re[5] = {4, 8, 8, 8, 8};
         bool pr[5] = {true, true, true, true, true};
-        if (use_tma && scalar_tma_args(rp, re, pr, &ta)) {
+        if (use_tma && scalar_tma_args(rp, re, pr, 2048, &ta)) {
             for (int j = 0; j < 3; ++j) { ta.lo[j] = lo[j]; ta.hi[j] = hi[j]; }
             ta.fcmp[0] = ta.fcmp[1] = -1;
             ta.fc[0] = ta.fc[1] = 0;
             ta.n = n;
-            if (mode) e = launch_scalar_tma<1, 3, true, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
-            else e = launch_scalar_tma<0, 3, true, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
-        } else if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
-        else e = launch_scalar<0, true, true, true>(sa, ws, o, m, s, nl);
+            if (mode) e = launch_scalar_tma<1, 3, true, 2048, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
+            else e = launch_scalar_tma<0, 3, true, 2048, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
+            set_fragment("scalar_tma");
+        } else {
+            if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
+            else e = launch_scalar<0, true, true, true>(sa, ws, o, m, s, nl);
+            set_fragment("scalar_ldg");
+        }
+    } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && va == fcol[0] && al16(cols[va].data) && use_tma &&
+               f32_interval(fcmp, fc, &sslo, &sshi)) {
+        SelSumArgs ss;
+        ss.v = (const float*)cols[va].data;
+        ss.lo = sslo;
+        ss.hi = sshi;
+        ss.n = n;
+        ss.nstages = SS_MAXSTAGES;
+        const int grid = num_sms();
+        unsigned int* dn = (unsigned int*)ws;
+        Slot16* parts = (Slot16*)((char*)ws + 256);
+        e = cudaMemsetAsync(dn, 0, 4, s);
+        if (e == cudaSuccess) {
+            const size_t smem = (size_t)ss.nstages * SS_TILE * 4 + 2 * ss.nstages * 8;
+            if (mode) {
+                cudaFuncSetAttribute(k_pipe_selsum_tma<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+                k_pipe_selsum_tma<1><<<grid, SCT_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
+            } else {
+                cudaFuncSetAttribute(k_pipe_selsum_tma<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+                k_pipe_selsum_tma<0><<<grid, SCT_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
+            }
+            ++*nl;
+            e = cudaGetLastError();
+        }
+        set_fragment("selsum_tma");
     } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && al16(cols[fcol[0]].data)) {
         // selective aggregation over one f32 column (Fig 15 / C1)
         ScalarArgs<float, float, float, float, float> sa;
@@ -1412,19 +1867,143 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
         const void* rp[5] = {sa.f0, nullptr, nullptr, sa.va, nullptr};
         const int re[5] = {4, 4, 4, 4, 4};
         bool pr[5] = {true, false, false, true, false};
-        if (use_tma && scalar_tma_args(rp, re, pr, &ta)) {
+        if (use_tma && scalar_tma_args(rp, re, pr, 8192, &ta)) {
             for (int j = 0; j < 3; ++j) { ta.lo[j] = lo[j]; ta.hi[j] = hi[j]; }
             ta.fcmp[0] = fcmp[0]; ta.fcmp[1] = fcmp[1];
             ta.fc[0] = fc[0]; ta.fc[1] = fc[1];
             ta.n = n;
-            if (mode) e = launch_scalar_tma<1, 1, false, float, float, float, float, float>(ta, ws, o, m, s, nl);
-            else e = launch_scalar_tma<0, 1, false, float, float, float, float, float>(ta, ws, o, m, s, nl);
-        } else if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
-        else e = launch_scalar<0, false, false, false>(sa, ws, o, m, s, nl);
+            if (mode) e = launch_scalar_tma<1, 1, false, 8192, float, float, float, float, float>(ta, ws, o, m, s, nl);
+            else e = launch_scalar_tma<0, 1, false, 8192, float, float, float, float, float>(ta, ws, o, m, s, nl);
+            set_fragment("scalar_tma");
+        } else {
+            if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
+            else e = launch_scalar<0, false, false, false>(sa, ws, o, m, s, nl);
+            set_fragment("scalar_ldg");
+        }
     } else {
         return VD_OK;
     }
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    *done = true;
+    return VD_OK;
+}
+
+// ---- gather-fold matching -------------------------------------------------------
+static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                        void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    const char* var = getenv("VD_GF_VARIANT");
+    if (var && strcmp(var, "off") == 0) return VD_OK;
+    if (ncols > GF_MAXCOLS || p->ngroups > 512) return VD_OK;
+    const int nref = ncols + p->ngathers;
+    auto dtype_of = [&](int c) { return c < ncols ? cols[c].dtype : dims[p->gathers[c - ncols].dim_col].dtype; };
+    auto is_int = [](int dt) { return dt == VD_U8 || dt == VD_I32 || dt == VD_I64; };
+    GfArgs A;
+    std::memset(&A, 0, sizeof(A));
+    // staged columns: all base columns (16B aligned, integer)
+    int off = 0;
+    for (int c = 0; c < ncols; ++c) {
+        if (((uintptr_t)cols[c].data % 16) != 0) return VD_OK;
+        A.col[c] = cols[c].data;
+        A.dt[c] = cols[c].dtype;
+        A.esz[c] = (int)dtype_size(cols[c].dtype);
+        A.soff[c] = off;
+        off += GF_TILE * A.esz[c];
+    }
+    A.ncols = ncols;
+    A.stage_bytes = off;
+    // gathers
+    A.ngathers = p->ngathers;
+    for (int g = 0; g < p->ngathers; ++g) {
+        const vd_column& d = dims[p->gathers[g].dim_col];
+        if (!is_int(d.dtype) || !is_int(cols[p->gathers[g].fk_col].dtype)) return VD_OK;
+        A.g_fk[g] = p->gathers[g].fk_col;
+        A.g_bias[g] = p->gathers[g].bias;
+        A.g_p[g] = d.data;
+        A.g_len[g] = d.len;
+        A.g_dt[g] = d.dtype;
+    }
+    // predicate, base terms first within each conjunction
+    vd_pred pr = p->pred;
+    for (int c = 0; c < pr.nconj; ++c) {
+        vd_conj& cj = pr.conj[c];
+        vd_term tmp[VD_MAX_TERMS];
+        int k = 0;
+        for (int t = 0; t < cj.nterms; ++t) if (cj.terms[t].col < ncols) tmp[k++] = cj.terms[t];
+        A.nbase[c] = k;
+        for (int t = 0; t < cj.nterms; ++t) if (cj.terms[t].col >= ncols) tmp[k++] = cj.terms[t];
+        for (int t = 0; t < cj.nterms; ++t) cj.terms[t] = tmp[t];
+    }
+    make_devpred(&pr, &A.pred);
+    // key
+    A.nkey = p->nkeyparts;
+    int64_t ylo = 0, yhi = -1;
+    for (int k = 0; k < p->nkeyparts; ++k) {
+        const vd_keypart& kp = p->key[k];
+        if (!is_int(dtype_of(kp.col))) return VD_OK;
+        A.k_col[k] = kp.col;
+        A.k_fn[k] = kp.fn;
+        A.k_sub[k] = kp.sub;
+        A.k_mult[k] = kp.mult;
+        if (kp.fn == 1) {
+            const vd_column* kc = kp.col < ncols ? &cols[kp.col] : &dims[p->gathers[kp.col - ncols].dim_col];
+            if (kc->has_minmax && kc->max - kc->min < GF_MAXYEARDAYS) { ylo = kc->min; yhi = kc->max; }
+        }
+    }
+    A.year_lo = (int32_t)ylo;
+    A.year_days = (int32_t)(yhi - ylo + 1);
+    A.ngroups = (int32_t)p->ngroups;
+    // aggregates: SUM of int64 products or COUNT; exactness from metadata
+    int grid = num_sms();
+    double rows_per_warp = std::ceil((double)n / ((double)grid * GF_CW)) + GF_TILE;
+    A.naggs = p->naggs;
+    for (int g = 0; g < p->naggs; ++g) {
+        const vd_agg& ag = p->aggs[g];
+        A.a_kind[g] = ag.kind;
+        if (ag.kind == VD_AGG_COUNT) continue;
+        if (ag.kind != VD_AGG_SUM) return VD_OK;
+        A.a_nf[g] = ag.nfactors;
+        double mx = 1;
+        for (int f = 0; f < ag.nfactors; ++f) {
+            A.a_col[g][f] = ag.f[f].col;
+            A.a_a[g][f] = ag.f[f].a;
+            A.a_b[g][f] = ag.f[f].b;
+            if (ag.f[f].col < 0) { mx *= std::fabs((double)ag.f[f].a); continue; }
+            if (!is_int(dtype_of(ag.f[f].col))) return VD_OK;
+            Bound b = col_bound(p, cols, ncols, dims, ag.f[f].col);
+            if (!b.known) return VD_OK;
+            mx *= factor_absmax(ag.f[f], b);
+        }
+        if (mx * rows_per_warp >= 9.0e18) return VD_OK;
+    }
+    A.n = n;
+    // shared memory: ring + warp slots + staging + calendar + barriers
+    const int NS = (int)p->ngroups * (p->naggs + 1);
+    size_t fixed = (size_t)GF_CW * NS * 8 + (size_t)GF_CW * 32 * (p->naggs + 1) * 8 +
+                   (size_t)((A.year_days + 7) & ~7) * 2 + 2 * GF_MAXSTAGES * 8;
+    const size_t budget = 200 * 1024;
+    if (fixed + 2 * (size_t)off > budget) return VD_OK;
+    int ns = (int)((budget - fixed) / (size_t)off);
+    A.nstages = ns < 2 ? 2 : (ns > GF_MAXSTAGES ? GF_MAXSTAGES : ns);
+    size_t smem = fixed + (size_t)A.nstages * off;
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    Slot16* rawp = (Slot16*)out;
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    const int mode = p->sel_mode == VD_SEL_PREDICATED ? 1 : 0;
+    if (mode) {
+        cudaFuncSetAttribute(k_pipe_gf<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_gf<1><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
+    } else {
+        cudaFuncSetAttribute(k_pipe_gf<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_gf<0><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
+    }
+    ++*nl;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    (void)nref;
+    set_fragment("gather_fold");
     *done = true;
     return VD_OK;
 }
@@ -1519,12 +2098,15 @@ static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int nc
     ++*nl;
     e = cudaGetLastError();
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    set_fragment("generic");
     return VD_OK;
 }
 
 vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncols, int64_t n, const vd_column* dims,
                        int32_t, void* out, void* ws, size_t, cudaStream_t s, int* nl) {
+    set_fragment("");
     if (n == 0) {
+        set_fragment("empty");
         cudaError_t e = cudaMemsetAsync(out, 0, (size_t)p->ngroups * (p->naggs + 1) * 16, s);
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
         return VD_OK;
@@ -1534,6 +2116,8 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         vd_status st = try_q1(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+        st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
     }
     return run_generic(p, cols, ncols, n, dims, out, ws, s, nl);

@@ -180,6 +180,19 @@ __global__ void __launch_bounds__(SCAN_THREADS) k_scan_i32(const int32_t* __rest
     }
 }
 
+size_t scan_ws_bytes(int64_t m) { return 256 + ((((size_t)(m + SCAN_TILE - 1) / SCAN_TILE) * 8 + 255) & ~(size_t)255); }
+
+cudaError_t launch_scan_i32(const int32_t* in, int64_t m, int64_t* out, void* ws, cudaStream_t s, int* nl) {
+    if (m <= 0) return cudaSuccess;
+    int64_t st = (m + SCAN_TILE - 1) / SCAN_TILE;
+    cudaError_t e = cudaMemsetAsync(ws, 0, 256 + (size_t)st * 8, s);
+    if (e != cudaSuccess) return e;
+    int sg = (int)(st < (int64_t)num_sms() * 4 ? st : (int64_t)num_sms() * 4);
+    k_scan_i32<<<sg, SCAN_THREADS, 0, s>>>(in, m, out, (uint64_t*)((char*)ws + 256), (unsigned long long*)ws, st);
+    ++*nl;
+    return cudaGetLastError();
+}
+
 template <typename T>
 __global__ void __launch_bounds__(PART_THREADS) k_part_place(const T* __restrict__ v, int64_t n, int64_t from, int npiv,
                                                              int64_t tw, int64_t ntiles,

@@ -19,6 +19,9 @@
 //                        the next step.  The valid prefix is then streamed
 //                        out with coalesced stores.  No lane of one store
 //                        instruction shares an address with another.
+#include <cstdlib>
+#include <cstring>
+
 #include "vd_common.cuh"
 #include "vd_internal.h"
 #include "vd_lookback.cuh"
@@ -33,15 +36,18 @@ constexpr int SEL_WROWS = SEL_CH * 128;            // rows per warp per tile
 constexpr int SEL_TILE = SEL_WARPS * SEL_WROWS;    // 4096 rows per tile
 
 // ---- flag providers: flags of 4 consecutive rows starting at row0 ----------
+struct NoRaw {};
+
 struct GenericFlags {
     DevPred P;
     DevCols C;
+    typedef NoRaw Raw;
+    __device__ __forceinline__ void load(int64_t, int64_t, Raw&) const {}
+    __device__ __forceinline__ void eval(const Raw&, int64_t row0, int64_t n, bool f[4]) const { flags4(row0, n, f); }
+    __device__ __forceinline__ bool eval1(int64_t r, int64_t n) const { return (r < n) && eval_pred_row(P, C, r); }
     __device__ __forceinline__ void flags4(int64_t row0, int64_t n, bool f[4]) const {
 #pragma unroll
-        for (int j = 0; j < 4; ++j) {
-            int64_t r = row0 + j;
-            f[j] = (r < n) && eval_pred_row(P, C, r);
-        }
+        for (int j = 0; j < 4; ++j) f[j] = eval1(row0 + j, n);
     }
 };
 
@@ -92,6 +98,22 @@ struct TermFlags {
         if (IsFloat<T>::value) return cmp_flt(cmp, (double)x, fv);
         return cmp_int(cmp, (int64_t)x, iv);
     }
+    // raw values of 4 rows, loaded ahead of their evaluation (software pipelining)
+    struct Raw {
+        T v[4];
+    };
+    __device__ __forceinline__ void load(int64_t row0, int64_t n, Raw& r) const {
+        if (ALIGNED && row0 + 4 <= n) {
+            Vec4Load<T>::ld(p + row0, r.v);
+        } else {
+#pragma unroll
+            for (int j = 0; j < 4; ++j) r.v[j] = (row0 + j < n) ? __ldg(p + row0 + j) : T(0);
+        }
+    }
+    __device__ __forceinline__ void eval(const Raw& r, int64_t row0, int64_t n, bool f[4]) const {
+#pragma unroll
+        for (int j = 0; j < 4; ++j) f[j] = (row0 + j < n) && test(r.v[j]);
+    }
     __device__ __forceinline__ void flags4(int64_t row0, int64_t n, bool f[4]) const {
         T v[4];
         if (ALIGNED && row0 + 4 <= n) {
@@ -114,6 +136,9 @@ struct HeadFlags {
     const void* mat;
     int32_t dt;
     int64_t from, num, den, cap;
+    typedef NoRaw Raw;
+    __device__ __forceinline__ void load(int64_t, int64_t, Raw&) const {}
+    __device__ __forceinline__ void eval(const Raw&, int64_t row0, int64_t n, bool f[4]) const { flags4(row0, n, f); }
     __device__ __forceinline__ int64_t value(int64_t i) const {
         if (mat) return dt == VD_I32 ? (int64_t)__ldg((const int32_t*)mat + i) : (int64_t)__ldg((const long long*)mat + i);
         i128 q = ((i128)i * num) / den;
@@ -121,123 +146,340 @@ struct HeadFlags {
         if (cap != 0) v %= cap;
         return (int64_t)v;
     }
+    __device__ __forceinline__ bool eval1(int64_t r, int64_t n) const {
+        return (r < n) && (r == 0 || value(r) != value(r - 1));
+    }
     __device__ __forceinline__ void flags4(int64_t row0, int64_t n, bool f[4]) const {
 #pragma unroll
-        for (int j = 0; j < 4; ++j) {
-            int64_t r = row0 + j;
-            f[j] = (r < n) && (r == 0 || value(r) != value(r - 1));
-        }
+        for (int j = 0; j < 4; ++j) f[j] = eval1(row0 + j, n);
     }
 };
 
+// One tile of the selection: flags -> ranks -> look-back -> positions.
+template <int MODE, class F>
+__device__ __forceinline__ void select_tile(const F& fl, const typename F::Raw (&raw)[SEL_CH], int64_t tile,
+                                            int64_t n, int32_t* __restrict__ out, int64_t* __restrict__ out_count,
+                                            uint64_t* __restrict__ status, int64_t ntiles, int64_t* s_base,
+                                            int* s_wtot, int* s_woff, int32_t* s_stage) {
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const unsigned lt = lanemask_lt();
+    const int64_t row_w = tile * SEL_TILE + (int64_t)warp * SEL_WROWS;
+    unsigned fm = 0;  // bit k*4+j: row row_w + k*128 + lane*4 + j qualifies
+#pragma unroll
+    for (int k = 0; k < SEL_CH; ++k) {
+        bool f[4];
+        fl.eval(raw[k], row_w + k * 128 + lane * 4, n, f);
+#pragma unroll
+        for (int j = 0; j < 4; ++j) fm |= (f[j] ? 1u : 0u) << (k * 4 + j);
+    }
+    unsigned b[SEL_CH][4];
+    int ck[SEL_CH];
+    int wtot = 0;
+#pragma unroll
+    for (int k = 0; k < SEL_CH; ++k) {
+        ck[k] = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            b[k][j] = __ballot_sync(VD_FULL, (fm >> (k * 4 + j)) & 1u);
+            ck[k] += __popc(b[k][j]);
+        }
+        wtot += ck[k];
+    }
+    if (lane == 0) s_wtot[warp] = wtot;
+    __syncthreads();
+    if (warp == 0) {
+        int v = lane < SEL_WARPS ? s_wtot[lane] : 0;
+        int incl = v;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            int u = __shfl_up_sync(VD_FULL, incl, o);
+            if (lane >= o) incl += u;
+        }
+        if (lane < SEL_WARPS) s_woff[lane] = incl - v;
+        int64_t agg = __shfl_sync(VD_FULL, incl, SEL_WARPS - 1);
+        int64_t base = lookback_exclusive_w128(status, tile, agg, lane);
+        if (lane == 0) {
+            *s_base = base;
+            if (tile == ntiles - 1) *out_count = base + agg;
+        }
+    }
+    __syncthreads();
+    const int64_t base = *s_base + s_woff[warp];
+
+    if (MODE == 0) {
+        int cur = 0;
+#pragma unroll
+        for (int k = 0; k < SEL_CH; ++k) {
+            int before = 0;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) before += __popc(b[k][j] & lt);
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                if ((fm >> (k * 4 + j)) & 1u) {
+                    out[base + cur + before] = (int32_t)(row_w + k * 128 + lane * 4 + j);
+                    ++before;
+                }
+            }
+            cur += ck[k];
+        }
+    } else {
+        int32_t* st = s_stage + warp * SEL_WROWS;
+        int cur = 0;
+#pragma unroll
+        for (int k = 0; k < SEL_CH; ++k) {
+            int sel_before = 0;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) sel_before += __popc(b[k][j] & lt);
+            int item_before = lane * 4;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                int f = (fm >> (k * 4 + j)) & 1u;
+                int addr = cur + (f ? sel_before : ck[k] + (item_before - sel_before));
+                st[addr] = (int32_t)(row_w + k * 128 + lane * 4 + j);  // unconditional write
+                sel_before += f;                                         // cursor += predicate
+                ++item_before;
+            }
+            cur += ck[k];
+            __syncwarp();
+        }
+        for (int i = lane; i < wtot; i += 32) out[base + i] = st[i];
+        __syncwarp();
+    }
+}
+
+// Persistent CTAs, tiles claimed in order from an atomic counter, two tiles
+// per CTA in flight: the next tile's loads are issued before the current
+// tile's look-back, so HBM stays busy while the look-back waits on L2.
 template <int MODE, class F>
 __global__ void __launch_bounds__(SEL_THREADS) k_select(F fl, int64_t n, int32_t* __restrict__ out,
                                                         int64_t* __restrict__ out_count, uint64_t* __restrict__ status,
                                                         unsigned long long* __restrict__ tile_ctr, int64_t ntiles) {
-    __shared__ int64_t s_tile;
+    __shared__ int64_t s_next;
     __shared__ int64_t s_base;
     __shared__ int s_wtot[SEL_WARPS];
     __shared__ int s_woff[SEL_WARPS];
     __shared__ int32_t s_stage[MODE == 1 ? SEL_WARPS * SEL_WROWS : 1];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const unsigned lt = lanemask_lt();
+    typename F::Raw ra[SEL_CH], rb[SEL_CH];
 
-    for (;;) {
-        if (threadIdx.x == 0) s_tile = (int64_t)atomicAdd(tile_ctr, 1ull);
+    auto claim = [&]() -> int64_t {
+        if (threadIdx.x == 0) s_next = (int64_t)atomicAdd(tile_ctr, 1ull);
         __syncthreads();
-        const int64_t tile = s_tile;
-        if (tile >= ntiles) break;
+        int64_t t = s_next;
+        __syncthreads();
+        return t;
+    };
+    auto load = [&](int64_t tile, typename F::Raw (&r)[SEL_CH]) {
         const int64_t row_w = tile * SEL_TILE + (int64_t)warp * SEL_WROWS;
+#pragma unroll
+        for (int k = 0; k < SEL_CH; ++k) fl.load(row_w + k * 128 + lane * 4, n, r[k]);
+    };
+    int64_t cur = claim();
+    if (cur < ntiles) load(cur, ra);
+    for (;;) {
+        if (cur >= ntiles) break;
+        int64_t nxt = claim();
+        if (nxt < ntiles) load(nxt, rb);
+        select_tile<MODE>(fl, ra, cur, n, out, out_count, status, ntiles, &s_base, s_wtot, s_woff, s_stage);
+        cur = nxt;
+        if (cur >= ntiles) break;
+        nxt = claim();
+        if (nxt < ntiles) load(nxt, ra);
+        select_tile<MODE>(fl, rb, cur, n, out, out_count, status, ntiles, &s_base, s_wtot, s_woff, s_stage);
+        cur = nxt;
+    }
+}
 
-        unsigned fm = 0;  // bit k*4+j: row row_w + k*128 + lane*4 + j qualifies
+// ---- bitmap selection ---------------------------------------------------------------
+// Fig 8: a `break` materialises the predicate data-parallel, and
+// foldSelect then emits the positions.  Here the materialised predicate is a
+// bitmap (1 bit per row; 125 MB for 1e9 rows, largely L2-resident) with a
+// population count per 1024-row chunk:
+//   k_sel_bits_*  streaming pass: flags -> bitmap words + chunk counts
+//   scan          chunk counts -> chunk offsets (look-back scan)
+//   k_sel_write   positions from the bitmap: branching (each qualifying bit
+//                 stores its position) or predicated (cursor arithmetic:
+//                 every row of the chunk is written to a shared-memory stage,
+//                 qualifying rows at the cursor, the rest past it, then the
+//                 qualifying prefix streams out with coalesced stores).
+// No serial chain: each pass is fully data parallel, unlike a single-pass
+// look-back whose throughput is bounded by window x tile per L2 round trip.
+constexpr int BM_THREADS = 256;
+constexpr int BM_CHUNK = 1024;  // rows per warp chunk = 32 words
+
+// Bitmap layout ("ballot order"): chunk c holds rows c*1024 + q*128 + 4*L + j
+// (q = 0..7, lane L = 0..31, j = 0..3) as bit L of word c*32 + q*4 + j, so
+// every load instruction of the flag pass reads 512 contiguous bytes and
+// every word is one warp ballot.
+template <typename T, bool ALIGNED>
+__global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNED> fl, int64_t n,
+                                                             uint32_t* __restrict__ bits,
+                                                             int32_t* __restrict__ counts, int64_t nchunks) {
+    const int lane = threadIdx.x & 31;
+    const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
+    const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
+    for (int64_t c = gw; c < nchunks; c += nw) {
+        typename TermFlags<T, ALIGNED>::Raw raw[8];
 #pragma unroll
-        for (int k = 0; k < SEL_CH; ++k) {
+        for (int q = 0; q < 8; ++q) fl.load(c * BM_CHUNK + q * 128 + lane * 4, n, raw[q]);
+        uint32_t mine = 0;
+        int cnt = 0;
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
             bool f[4];
-            fl.flags4(row_w + k * 128 + lane * 4, n, f);
-#pragma unroll
-            for (int j = 0; j < 4; ++j) fm |= (f[j] ? 1u : 0u) << (k * 4 + j);
-        }
-        unsigned b[SEL_CH][4];
-        int ck[SEL_CH];
-        int wtot = 0;
-#pragma unroll
-        for (int k = 0; k < SEL_CH; ++k) {
-            ck[k] = 0;
+            fl.eval(raw[q], c * BM_CHUNK + q * 128 + lane * 4, n, f);
 #pragma unroll
             for (int j = 0; j < 4; ++j) {
-                b[k][j] = __ballot_sync(VD_FULL, (fm >> (k * 4 + j)) & 1u);
-                ck[k] += __popc(b[k][j]);
-            }
-            wtot += ck[k];
-        }
-        if (lane == 0) s_wtot[warp] = wtot;
-        __syncthreads();
-        if (warp == 0) {
-            int v = lane < SEL_WARPS ? s_wtot[lane] : 0;
-            int incl = v;
-#pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                int u = __shfl_up_sync(VD_FULL, incl, o);
-                if (lane >= o) incl += u;
-            }
-            if (lane < SEL_WARPS) s_woff[lane] = incl - v;
-            int64_t agg = __shfl_sync(VD_FULL, incl, SEL_WARPS - 1);
-            int64_t base = lookback_exclusive(status, tile, agg, lane);
-            if (lane == 0) {
-                s_base = base;
-                if (tile == ntiles - 1) *out_count = base + agg;
+                const uint32_t b = __ballot_sync(VD_FULL, f[j]);
+                cnt += __popc(b);
+                if (lane == q * 4 + j) mine = b;
             }
         }
-        __syncthreads();
-        const int64_t base = s_base + s_woff[warp];
+        bits[c * 32 + lane] = mine;
+        if (lane == 0) counts[c] = cnt;
+    }
+}
 
-        if (MODE == 0) {
-            int cur = 0;
+// Per-row predicates (several columns, run heads), same layout.
+template <class F>
+__global__ void __launch_bounds__(BM_THREADS) k_sel_bits_bal(F fl, int64_t n, uint32_t* __restrict__ bits,
+                                                             int32_t* __restrict__ counts, int64_t nchunks) {
+    const int lane = threadIdx.x & 31;
+    const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
+    const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
+    for (int64_t c = gw; c < nchunks; c += nw) {
+        uint32_t mine = 0;
+        int cnt = 0;
+#pragma unroll 2
+        for (int q = 0; q < 8; ++q) {
 #pragma unroll
-            for (int k = 0; k < SEL_CH; ++k) {
-                int before = 0;
-#pragma unroll
-                for (int j = 0; j < 4; ++j) before += __popc(b[k][j] & lt);
-#pragma unroll
-                for (int j = 0; j < 4; ++j) {
-                    if ((fm >> (k * 4 + j)) & 1u) {
-                        out[base + cur + before] = (int32_t)(row_w + k * 128 + lane * 4 + j);
-                        ++before;
-                    }
-                }
-                cur += ck[k];
+            for (int j = 0; j < 4; ++j) {
+                const uint32_t b = __ballot_sync(VD_FULL, fl.eval1(c * BM_CHUNK + q * 128 + lane * 4 + j, n));
+                cnt += __popc(b);
+                if (lane == q * 4 + j) mine = b;
             }
-        } else {
-            int32_t* st = s_stage + warp * SEL_WROWS;
-            int cur = 0;
+        }
+        bits[c * 32 + lane] = mine;
+        if (lane == 0) counts[c] = cnt;
+    }
+}
+
+__global__ void k_sel_total(const int64_t* __restrict__ offs, const int32_t* __restrict__ counts, int64_t nchunks,
+                            int64_t* __restrict__ out_count) {
+    *out_count = nchunks > 0 ? offs[nchunks - 1] + counts[nchunks - 1] : 0;
+}
+
+template <int MODE>
+__global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __restrict__ bits,
+                                                          const int64_t* __restrict__ offs, int64_t nchunks,
+                                                          int32_t* __restrict__ out) {
+    __shared__ int32_t s_stage[MODE == 1 ? (BM_THREADS / 32) * 128 : 1];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const unsigned lt = lanemask_lt();
+    const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
+    const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
+    for (int64_t c = gw; c < nchunks; c += nw) {
+        const uint32_t myword = bits[c * 32 + lane];
+        int64_t base = offs[c];
+        for (int q = 0; q < 8; ++q) {
+            uint32_t b[4];
+            int cnt = 0, before = 0, mine = 0;
 #pragma unroll
-            for (int k = 0; k < SEL_CH; ++k) {
-                int sel_before = 0;
+            for (int j = 0; j < 4; ++j) {
+                b[j] = __shfl_sync(VD_FULL, myword, q * 4 + j);
+                cnt += __popc(b[j]);
+                before += __popc(b[j] & lt);
+                mine += (b[j] >> lane) & 1u;
+            }
+            const int32_t row = (int32_t)(c * BM_CHUNK + q * 128 + lane * 4);
+            if (MODE == 0) {
+                // branching: a qualifying row stores its position (lanes of a
+                // store instruction write increasing, nearly contiguous slots)
+                int k = before;
 #pragma unroll
-                for (int j = 0; j < 4; ++j) sel_before += __popc(b[k][j] & lt);
-                int item_before = lane * 4;
+                for (int j = 0; j < 4; ++j)
+                    if ((b[j] >> lane) & 1u) out[base + k++] = row + j;
+            } else {
+                // predicated (cursor arithmetic): every row of the 128-row block
+                // is written; qualifying rows at the cursor, the others past it
+                int32_t* st = s_stage + warp * 128;
+                int sel = before, unsel = cnt + (lane * 4 - before);
 #pragma unroll
                 for (int j = 0; j < 4; ++j) {
-                    int f = (fm >> (k * 4 + j)) & 1u;
-                    int addr = cur + (f ? sel_before : ck[k] + (item_before - sel_before));
-                    st[addr] = (int32_t)(row_w + k * 128 + lane * 4 + j);  // unconditional write
-                    sel_before += f;                                         // cursor += predicate
-                    ++item_before;
+                    const int f = (b[j] >> lane) & 1u;
+                    st[f ? sel : unsel] = row + j;
+                    sel += f;
+                    unsel += 1 - f;
                 }
-                cur += ck[k];
+                __syncwarp();
+                for (int k = lane; k < cnt; k += 32) out[base + k] = st[k];
                 __syncwarp();
             }
-            for (int i = lane; i < wtot; i += 32) out[base + i] = st[i];
-            __syncwarp();
+            (void)mine;
+            base += cnt;
         }
-        __syncthreads();
     }
+}
+
+struct BmLayout {
+    int64_t nchunks;
+    uint32_t* bits;
+    int32_t* counts;
+    int64_t* offs;
+    void* scan_ws;
+};
+static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
+static BmLayout bm_layout(int64_t n, void* ws) {
+    BmLayout L;
+    L.nchunks = (n + BM_CHUNK - 1) / BM_CHUNK;
+    char* w = (char*)ws;
+    L.bits = (uint32_t*)w;
+    w += al256((size_t)L.nchunks * 32 * 4);
+    L.counts = (int32_t*)w;
+    w += al256((size_t)L.nchunks * 4);
+    L.offs = (int64_t*)w;
+    w += al256((size_t)L.nchunks * 8);
+    L.scan_ws = w;
+    return L;
+}
+static size_t bm_ws_bytes(int64_t n) {
+    int64_t nc = (n + BM_CHUNK - 1) / BM_CHUNK;
+    return al256((size_t)nc * 32 * 4) + al256((size_t)nc * 4) + al256((size_t)nc * 8) + scan_ws_bytes(nc) + 256;
+}
+static int bm_grid(int64_t nchunks) {
+    int64_t g = (int64_t)num_sms() * 8;
+    int64_t need = (nchunks * 32 + BM_THREADS - 1) / BM_THREADS;
+    if (g > need) g = need;
+    return (int)(g < 1 ? 1 : g);
+}
+
+template <int MODE, class LaunchBits>
+static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t* out_pos, int64_t* out_count,
+                                     void* ws, cudaStream_t s, int* nl) {
+    BmLayout L = bm_layout(n, ws);
+    if (L.nchunks == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
+    launch_bits(L, bm_grid(L.nchunks));
+    ++*nl;
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) return e;
+    if ((e = launch_scan_i32(L.counts, L.nchunks, L.offs, L.scan_ws, s, nl)) != cudaSuccess) return e;
+    k_sel_total<<<1, 1, 0, s>>>(L.offs, L.counts, L.nchunks, out_count);
+    k_sel_write<MODE><<<bm_grid(L.nchunks), BM_THREADS, 0, s>>>(L.bits, L.offs, L.nchunks, out_pos);
+    *nl += 2;
+    return cudaGetLastError();
 }
 
 size_t select_ws_bytes(int64_t n) {
     int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
     size_t b = 256 + (size_t)ntiles * 8;
-    return (b + 255) & ~(size_t)255;
+    size_t lb = (b + 255) & ~(size_t)255;
+    size_t bm = bm_ws_bytes(n);
+    return lb > bm ? lb : bm;
+}
+
+static bool use_lookback() {
+    const char* v = getenv("VD_SELECT_VARIANT");
+    return v && strcmp(v, "lookback") == 0;
 }
 
 static int select_grid(int64_t ntiles) {
@@ -267,10 +509,20 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
     bool aligned = ((uintptr_t)p % vecbytes) == 0;
     if (aligned) {
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv};
-        return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+        if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+        return run_select_bitmap<MODE>(
+            [&](const BmLayout& L, int grid) {
+                k_sel_bits_vec<T, true><<<grid, BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+            },
+            n, out_pos, out_count, ws, s, nl);
     }
     TermFlags<T, false> f{(const T*)p, t.cmp, t.iv, t.fv};
-    return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+    if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+    return run_select_bitmap<MODE>(
+        [&](const BmLayout& L, int grid) {
+            k_sel_bits_vec<T, false><<<grid, BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+        },
+        n, out_pos, out_count, ws, s, nl);
 }
 
 template <int MODE>
@@ -288,7 +540,12 @@ static cudaError_t select_mode(const DevCols& cols, const DevPred& pred, int64_t
         }
     }
     GenericFlags g{pred, cols};
-    return run_select<MODE>(g, n, out_pos, out_count, ws, s, nl);
+    if (use_lookback()) return run_select<MODE>(g, n, out_pos, out_count, ws, s, nl);
+    return run_select_bitmap<MODE>(
+        [&](const BmLayout& L, int grid) {
+            k_sel_bits_bal<GenericFlags><<<grid, BM_THREADS, 0, s>>>(g, n, L.bits, L.counts, L.nchunks);
+        },
+        n, out_pos, out_count, ws, s, nl);
 }
 
 cudaError_t launch_select(int mode, const DevCols& cols, const DevPred& pred, int64_t n, int32_t* out_pos,
@@ -300,7 +557,12 @@ cudaError_t launch_select(int mode, const DevCols& cols, const DevPred& pred, in
 cudaError_t launch_select_heads(const CtrlInfo& ci, int64_t n, int32_t* out_pos, int64_t* out_count, void* ws,
                                 size_t, cudaStream_t s, int* nl) {
     HeadFlags h{ci.mat, ci.mat_dtype, ci.from, ci.num, ci.den, ci.cap};
-    return run_select<0>(h, n, out_pos, out_count, ws, s, nl);
+    if (use_lookback()) return run_select<0>(h, n, out_pos, out_count, ws, s, nl);
+    return run_select_bitmap<0>(
+        [&](const BmLayout& L, int grid) {
+            k_sel_bits_bal<HeadFlags><<<grid, BM_THREADS, 0, s>>>(h, n, L.bits, L.counts, L.nchunks);
+        },
+        n, out_pos, out_count, ws, s, nl);
 }
 
 // out_run_off[r] = number of selected positions before run r's first row

@@ -16,10 +16,12 @@ namespace vd {
 
 static thread_local std::string t_err;
 static thread_local int t_launches = 0;
+static thread_local const char* t_fragment = "";
 
 void set_error(const std::string& msg) { t_err = msg; }
 void count_launches(int k) { t_launches += k; }
 void reset_launches() { t_launches = 0; }
+void set_fragment(const char* name) { t_fragment = name; }
 
 size_t dtype_size(int32_t dt) {
     switch (dt) {
@@ -280,6 +282,7 @@ const char* vd_status_str(vd_status s) {
 const char* vd_last_error(void) { return t_err.c_str(); }
 const char* vd_version(void) { return "voodoo-b200 0.1 (sm_100a)"; }
 int32_t vd_last_launch_count(void) { return t_launches; }
+const char* vd_last_fragment(void) { return t_fragment; }
 
 int32_t vd_abi_struct_sizes(size_t* out, int32_t n) {
     const size_t v[8] = {sizeof(vd_column), sizeof(vd_ctrl), sizeof(vd_term), sizeof(vd_conj),

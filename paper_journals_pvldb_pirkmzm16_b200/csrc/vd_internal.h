@@ -16,6 +16,7 @@ namespace vd {
 void set_error(const std::string& msg);
 void count_launches(int k);
 void reset_launches();
+void set_fragment(const char* name);
 
 size_t dtype_size(int32_t dt);
 
@@ -53,6 +54,10 @@ struct DevCols {
 void make_devpred(const vd_pred* p, DevPred* d);
 
 // ---- launchers (implemented in the .cu files); return cudaError_t ---------
+// k_scatter.cu: exclusive scan of int32 counts into int64 offsets (look-back)
+size_t scan_ws_bytes(int64_t m);
+cudaError_t launch_scan_i32(const int32_t* in, int64_t m, int64_t* out, void* ws, cudaStream_t s, int* nl);
+
 // k_select.cu
 size_t select_ws_bytes(int64_t n);
 cudaError_t launch_select(int mode, const DevCols& cols, const DevPred& pred, int64_t n, int32_t* out_pos,

@@ -122,6 +122,7 @@ _sigs = {
     "vd_merge_partials": (c_int32, [_P(vd_pipeline), _P(vd_column), c_int32, _P(vd_column), c_int32,
                                     _P(c_void_p), c_int32, c_void_p]),
     "vd_last_launch_count": (c_int32, []),
+    "vd_last_fragment": (ctypes.c_char_p, []),
     "vd_abi_struct_sizes": (c_int32, [_P(c_size_t), c_int32]),
 }
 EXPORTS = sorted(_sigs)
@@ -161,6 +162,11 @@ def version() -> str:
 
 def last_launch_count() -> int:
     return int(_L.vd_last_launch_count())
+
+
+def last_fragment() -> str:
+    """Name of the fragment the last run_pipeline on this thread ran."""
+    return _L.vd_last_fragment().decode()
 
 
 # ---- torch plumbing ---------------------------------------------------------------

@@ -1,0 +1,58 @@
+#!/usr/bin/env python
+"""Selectivity sweeps on one GPU (runs bench.py per point; one JSON line each).
+
+  python scripts/sweep.py fig1  > gpurun_out/sweep_fig1.jsonl   # C2: 1e9 f32 -> positions
+  python scripts/sweep.py fig15 > gpurun_out/sweep_fig15.jsonl  # selective aggregation (select + FoldSum)
+
+Fig 1 and Fig 15: branching vs
+predicated (cursor arithmetic) over selectivities 1..100 % (plus the Fig 15
+range down to 0.01 %).  Then `python scripts/sweep.py table FILE...` renders
+a markdown table for profiles/.
+"""
+import json
+import os
+import subprocess
+import sys
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+SEL = [0.0001, 0.001, 0.01, 0.05, 0.1, 0.2, 0.5, 0.8, 1.0]
+
+
+def run(workload, s, mode, steps):
+    cmd = [sys.executable, os.path.join(ROOT, "bench.py"), "--workload", workload, "--selectivity", str(s),
+           "--sel-mode", mode, "--steps", str(steps), "--no-cpu-baseline", "--no-e2e"]
+    out = subprocess.run(cmd, capture_output=True, text=True, timeout=600)
+    line = out.stdout.strip().splitlines()[-1] if out.stdout.strip() else "{}"
+    d = json.loads(line)
+    d["_sel"] = s
+    d["_mode"] = mode
+    return d
+
+
+def table(files):
+    rows = []
+    for f in files:
+        for ln in open(f):
+            if ln.strip():
+                rows.append(json.loads(ln))
+    print("| workload | selectivity | mode | ms | G rows/s | achieved GB/s | frac of measured |")
+    print("|---|---|---|---|---|---|---|")
+    for d in rows:
+        if "roofline" not in d:
+            continue
+        print(f"| {d['config']['workload']} | {d['_sel']} | {d['_mode']} | {d['ms_per_step']:.3f} | "
+              f"{d['value'] / 1e9:.1f} | {d['roofline']['achieved']:.0f} | {d['roofline']['frac']:.3f} |")
+
+
+def main():
+    what = sys.argv[1]
+    if what == "table":
+        return table(sys.argv[2:])
+    workload = {"fig1": "selpos", "fig15": "select"}[what]
+    for s in SEL:
+        for mode in ["branch", "predicated"]:
+            print(json.dumps(run(workload, s, mode, 30 if workload == "selpos" else 100)), flush=True)
+
+
+if __name__ == "__main__":
+    main()

@@ -27,11 +27,14 @@ def load(cols_np):
     return keep, views
 
 
-def run(plan, views, n, dims=()):
+def run(plan, views, n, dims=(), want=None):
     out = torch.empty(vd.partials_bytes(plan), dtype=torch.uint8, device="cuda")
     vd.run_pipeline(plan, views, n, dims, out=out)
     launches = vd.last_launch_count()
+    frag = vd.last_fragment()
     torch.cuda.synchronize()
+    if want is not None:
+        assert frag in want, (frag, want)
     return out.cpu().numpy().tobytes(), launches
 
 
@@ -48,12 +51,12 @@ def test_q1_vs_oracle(sel_mode, generic, n):
     exp = oracle.q1(li)
     keep, views = load([li[c] for c in plans.Q1_COLS])
     plan = plans.q1(sel_mode, force_generic=generic)
-    buf, nl = run(plan, views, n)
+    buf, nl = run(plan, views, n, want=("generic",) if generic else ("q1_tma",))
     got = vd.decode_partials(buf, plan)
     assert {k: v[:6] for k, v in got.items()} == exp
     for k, v in got.items():
         assert v[6] == v[5]  # row count slot == count(*) aggregate
-    assert nl == (1 if generic else 2)  # the Q1 fragment (+ remap) ran, not the generic one
+    assert nl == 1  # one fused kernel per pipeline call
 
 
 def test_q1_key_domain_proof_and_ship_edge():
@@ -97,13 +100,13 @@ def test_q6_vs_oracle(sel_mode, generic, n):
     rev, cnt = oracle.q6(li)
     keep, views = load([li[c] for c in plans.Q6_COLS])
     plan = plans.q6(sel_mode, force_generic=generic)
-    buf, nl = run(plan, views, n)
+    buf, nl = run(plan, views, n, want=("generic",) if generic else ("scalar_tma",))
     got = vd.decode_partials(buf, plan)
     if cnt == 0:
         assert got == {}
     else:
         assert got == {0: [rev, cnt, cnt]}
-    assert nl == (1 if generic else 2)
+    assert nl == 1
 
 
 @pytest.mark.parametrize("sel_mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED])
@@ -116,7 +119,7 @@ def test_selective_sum_f32_vs_oracle(sel_mode, generic, n):
     _, c, (sh, sl) = oracle.select_f32(v, t, "lt", want_positions=False)
     keep, views = load([v])
     plan = plans.selsum(t, sel_mode, force_generic=generic)
-    buf, nl = run(plan, views, n)
+    buf, nl = run(plan, views, n, want=("generic",) if generic else ("selsum_tma",))
     got = vd.decode_partials(buf, plan, float_aggs=[True, False])
     assert got[0][1] == c
     ref = sh + sl
@@ -137,28 +140,34 @@ def codes():
 
 
 @pytest.mark.parametrize("sel_mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED])
-def test_fkj_q19_vs_oracle(sel_mode):
+@pytest.mark.parametrize("generic", [False, True])
+@pytest.mark.parametrize("n", [None, 100003])
+def test_fkj_q19_vs_oracle(sel_mode, generic, n):
     sf = 0.05
-    li = lineitem(sf)
+    li = lineitem(sf, n)
     part, supp = _dims(sf)
     exp = oracle.fkj(0, li, part, supp)
     keep, views = load([li[c] for c in plans.Q19_COLS])
     dkeep, dviews = load([part[c] for c in plans.Q19_DIMS])
-    plan = plans.q19(codes(), sel_mode)
-    got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews)[0], plan)
+    plan = plans.q19(codes(), sel_mode, force_generic=generic)
+    got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews,
+                                 want=("generic",) if generic else ("gather_fold",))[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
 @pytest.mark.parametrize("sel_mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED])
-def test_fkj_q9_vs_oracle(sel_mode):
+@pytest.mark.parametrize("generic", [False, True])
+@pytest.mark.parametrize("n", [None, 100003])
+def test_fkj_q9_vs_oracle(sel_mode, generic, n):
     sf = 0.05
-    li = lineitem(sf)
+    li = lineitem(sf, n)
     part, supp = _dims(sf)
     exp = oracle.fkj(1, li, part, supp)
     keep, views = load([li[c] for c in plans.Q9_COLS])
     dkeep, dviews = load([supp[c] for c in plans.Q9_DIMS])
-    plan = plans.q9(sel_mode)
-    got = vd.decode_partials(run(plan, views, len(li["l_suppkey"]), dviews)[0], plan)
+    plan = plans.q9(sel_mode, force_generic=generic)
+    got = vd.decode_partials(run(plan, views, len(li["l_suppkey"]), dviews,
+                                 want=("generic",) if generic else ("gather_fold",))[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
@@ -208,3 +217,28 @@ def test_virtual_shards_merge_equals_whole_q1():
         merged = vd.merge_partials(plan, views, [], parts)
         got = vd.decode_partials(merged, plan)
         assert {k: v[:6] for k, v in got.items()} == exp
+
+
+@pytest.mark.parametrize("op", [">", ">=", "<", "<=", "=="])
+@pytest.mark.parametrize("c", [0.1, float(np.float32(0.5)), 0.75000000000000011])
+def test_selective_sum_f32_interval_edges(op, c):
+    """The f32 interval form of a single comparison against a double constant
+    (x > c <=> x >= succ(floor32(c)), ...) agrees with exact comparisons of
+    the f32 values promoted to double (numpy), including the f32 neighbours
+    of the constant, epsilon (NaN) and infinities."""
+    base = np.float32(c)
+    near = [np.nextafter(base, np.float32(-np.inf)), base, np.nextafter(base, np.float32(np.inf))]
+    v = np.concatenate([np.array(near * 5000, dtype=np.float32), gen.host(gen.F32_UNIFORM, 100003, seed=5),
+                        np.array([np.inf, -np.inf, np.nan, 0.0], dtype=np.float32)])
+    keep, views = load([v])
+    plan = vd.pipeline(pred_=vd.pred([[(0, op, float(c))]]), aggs=[("sum", [0]), ("count",)])
+    buf, _ = run(plan, views, len(v), want=("selsum_tma",))
+    got = vd.decode_partials(buf, plan, float_aggs=[True, False])
+    x = v.astype(np.float64)
+    m = {">": x > c, ">=": x >= c, "<": x < c, "<=": x <= c, "==": x == c}[op] & ~np.isnan(x)
+    if m.sum() == 0:
+        assert got == {}
+        return
+    assert got[0][1] == int(m.sum())
+    ref = float(np.sum(x[m]))
+    assert got[0][0] == ref or abs(got[0][0] - ref) <= 1e-9 * abs(ref)
