@@ -54,6 +54,8 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     ap.add_argument("--seed", type=int, default=0x5EEDC0DE)
+    ap.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
+                    help="process-group backend for N > 1 (gloo: test mode, ranks may share a GPU)")
     return ap.parse_args()
 
 
@@ -206,10 +208,10 @@ def main():
     import gen
     from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
 
-    torch.cuda.set_device(local)
-    dev = torch.device("cuda", local)
-    if world > 1:
-        dist.init_process_group("nccl", device_id=dev)
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % ndev)
+    dev = torch.device("cuda", local % ndev)
+    comm = Comm(world, args.dist_backend, dev)
     stream = torch.cuda.current_stream()
 
     w = args.workload
@@ -274,8 +276,7 @@ def main():
 
     def step():
         vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
-        if world > 1:
-            dist.all_gather_into_tensor(gathered, out)
+        comm.all_gather(out, gathered)
 
     steps = args.steps if args.steps is not None else (300 if w in ("q1", "q19", "q9") else 1000)
     for _ in range(max(args.warmup, 0)):
@@ -287,8 +288,7 @@ def main():
     clocks = ClockSampler(local)
     clocks.start()
     time.sleep(0.3)
-    if world > 1:
-        dist.barrier()
+    comm.barrier()
     torch.cuda.synchronize()
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(steps)]
     t_start = torch.cuda.Event(enable_timing=True)
@@ -299,20 +299,15 @@ def main():
         ev[i][0].record(stream)
         vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
         ev[i][1].record(stream)
-        if world > 1:
-            dist.all_gather_into_tensor(gathered, out)
+        comm.all_gather(out, gathered)
     t_end.record(stream)
     torch.cuda.synchronize()
-    if world > 1:
-        dist.barrier()
+    comm.barrier()
     wall = time.perf_counter() - wall0
     clk = clocks.stop()
     elapsed_ms = t_start.elapsed_time(t_end)
     kernel_ms = sum(s.elapsed_time(e) for s, e in ev) / steps
-    if world > 1:
-        tt = torch.tensor([elapsed_ms, kernel_ms], dtype=torch.float64, device=dev)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        elapsed_ms, kernel_ms = float(tt[0]), float(tt[1])
+    elapsed_ms, kernel_ms = comm.max([elapsed_ms, kernel_ms])
     ms_per_step = elapsed_ms / steps
 
     # result check (merge of the per-rank partials, host side)
@@ -327,7 +322,7 @@ def main():
     # ---- e2e: host buffers in, result out, through the public API -------------
     e2e = None
     if not args.no_e2e:
-        e2e = e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, dist, pbytes)
+        e2e = e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, comm, pbytes)
 
     peak, peak_kind = hbm_peak()
     bpr = BYTES_PER_ROW[w]
@@ -365,6 +360,8 @@ def main():
         "e2e": e2e,
         "gpu_launches": launches_per_step * steps,
         "result": {str(k): [str(x) for x in v] for k, v in list(result.items())[:8]},
+        "result_groups": len(result),
+        "result_digest": __import__("hashlib").sha256(repr(sorted(result.items())).encode()).hexdigest()[:16],
         "wall_s": wall,
     }
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -372,9 +369,7 @@ def main():
                                             args.selectivity)
     if rank == 0:
         print(json.dumps(line), flush=True)
-    if world > 1:
-        dist.barrier()
-        dist.destroy_process_group()
+    comm.close()
 
 
 def selpos_main(args, rank, world, local):
@@ -388,10 +383,10 @@ def selpos_main(args, rank, world, local):
     import gen
     from paper_journals_pvldb_pirkmzm16_b200 import vd
 
-    torch.cuda.set_device(local)
-    dev = torch.device("cuda", local)
-    if world > 1:
-        dist.init_process_group("nccl", device_id=dev)
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % ndev)
+    dev = torch.device("cuda", local % ndev)
+    comm = Comm(world, args.dist_backend, dev)
     stream = torch.cuda.current_stream()
     n_total = args.rows or 10**9
     a, b = rank * n_total // world, (rank + 1) * n_total // world
@@ -417,8 +412,7 @@ def selpos_main(args, rank, world, local):
     clocks = ClockSampler(local)
     clocks.start()
     time.sleep(0.3)
-    if world > 1:
-        dist.barrier()
+    comm.barrier()
     torch.cuda.synchronize()
     ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(steps)]
     for i in range(steps):
@@ -428,10 +422,7 @@ def selpos_main(args, rank, world, local):
     torch.cuda.synchronize()
     clk = clocks.stop()
     ms = sum(s.elapsed_time(e) for s, e in ev) / steps
-    if world > 1:
-        tt = torch.tensor([ms], dtype=torch.float64, device=dev)
-        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        ms = float(tt[0])
+    ms = comm.max([ms])[0]
     c = int(cnt.item())
     peak, kind = hbm_peak()
     alg = (4 * n + 4 * c) / (ms * 1e-3) / 1e9
@@ -446,8 +437,50 @@ def selpos_main(args, rank, world, local):
             "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
     if rank == 0:
         print(json.dumps(line), flush=True)
-    if world > 1:
-        dist.destroy_process_group()
+    comm.close()
+
+
+class Comm:
+    """The cross-rank plumbing of the bench (torch.distributed): NCCL over
+    NVLink on device tensors, or gloo on host copies (test mode: several
+    ranks may share one GPU)."""
+
+    def __init__(self, world, backend, dev):
+        import torch.distributed as dist
+        self.world, self.backend, self.dev, self.dist = world, backend, dev, dist
+        if world > 1:
+            if backend == "nccl":
+                dist.init_process_group("nccl", device_id=dev)
+            else:
+                dist.init_process_group("gloo")
+
+    def barrier(self):
+        if self.world > 1:
+            self.dist.barrier()
+
+    def all_gather(self, local, gathered):
+        if self.world == 1:
+            return
+        if self.backend == "nccl":
+            self.dist.all_gather_into_tensor(gathered, local)
+        else:
+            h = local.cpu()
+            g = gathered.new_empty(gathered.shape, device="cpu")
+            self.dist.all_gather_into_tensor(g, h)
+            gathered.copy_(g)
+
+    def max(self, vals):
+        if self.world == 1:
+            return vals
+        import torch
+        t = torch.tensor(vals, dtype=torch.float64, device=self.dev if self.backend == "nccl" else "cpu")
+        self.dist.all_reduce(t, op=self.dist.ReduceOp.MAX)
+        return [float(x) for x in t.tolist()]
+
+    def close(self):
+        if self.world > 1:
+            self.dist.barrier()
+            self.dist.destroy_process_group()
 
 
 def _dt(col):
@@ -457,7 +490,7 @@ def _dt(col):
             np.float64: "float64"}[gen.dtype_of(col)]
 
 
-def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, dist, pbytes):
+def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, stream, world, comm, pbytes):
     """Through the public API from pinned host buffers: vd_load_column (H2D)
     of every input column, vd_run_pipeline, D2H of the partials."""
     try:
@@ -474,8 +507,7 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
     ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
     reps = 3
     torch.cuda.synchronize()
-    if world > 1:
-        dist.barrier()
+    comm.barrier()
     t0 = time.perf_counter()
     for _ in range(reps):
         vcols = []
@@ -487,10 +519,7 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
         res.copy_(out, non_blocking=True)
         torch.cuda.synchronize()
     dt = (time.perf_counter() - t0) / reps
-    if world > 1:
-        t = torch.tensor([dt], dtype=torch.float64, device=dev)
-        dist.all_reduce(t, op=dist.ReduceOp.MAX)
-        dt = float(t[0])
+    dt = comm.max([dt])[0]
     h2d = sum(c.numel() * c.element_size() for c in cols)
     del host, dst
     return {"value": (n * world) / dt, "unit": "rows/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": pbytes,

@@ -1075,6 +1075,9 @@ struct GfArgs {
     // predicate: per conjunction, base terms first (nbase[c] of them)
     DevPred pred;
     int32_t nbase[VD_MAX_CONJ];
+    // base-column terms common to every conjunction, hoisted and tested first
+    int32_t ncommon;
+    DevTerm common[VD_MAX_TERMS];
     // key
     int32_t nkey;
     int32_t k_col[VD_MAX_KEYPARTS], k_fn[VD_MAX_KEYPARTS];
@@ -1129,6 +1132,8 @@ __device__ __forceinline__ Val gf_fetch(const GfArgs& a, const GfRow& w, int c) 
 }
 
 __device__ __forceinline__ bool gf_pred(const GfArgs& a, const GfRow& w) {
+    for (int k = 0; k < a.ncommon; ++k)
+        if (!term_true(a.common[k], gf_base(a, w, a.common[k].col))) return false;
     if (a.pred.nconj == 0) return true;
     // phase 1: base-column terms of every conjunction (no gathers)
     unsigned alive = 0;
@@ -1153,7 +1158,7 @@ __device__ __forceinline__ bool gf_pred(const GfArgs& a, const GfRow& w) {
     return false;
 }
 
-template <int MODE>
+template <int MODE, bool SCALAR>
 __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant__ GfArgs a, int64_t ntiles,
                                                            Slot16* __restrict__ parts, unsigned int* __restrict__ done,
                                                            Slot16* __restrict__ out) {
@@ -1176,8 +1181,31 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
     for (int k = threadIdx.x; k < a.year_days; k += GF_THREADS) ytab[k] = (int16_t)year_of_day(a.year_lo + k);
     __syncthreads();
 
+    int64_t racc[VD_MAX_AGGS + 1];  // SCALAR: per-thread accumulators (one group)
+#pragma unroll
+    for (int g = 0; g <= VD_MAX_AGGS; ++g) racc[g] = 0;
     auto process = [&](const GfRow& w, bool valid) {
         bool ok = valid && gf_pred(a, w);
+        if (SCALAR) {
+            if (ok) {
+#pragma unroll
+                for (int g = 0; g < VD_MAX_AGGS; ++g) {
+                    if (g >= NA) break;
+                    int64_t pr = 1;
+                    if (a.a_kind[g] != VD_AGG_COUNT) {
+                        for (int f = 0; f < a.a_nf[g]; ++f) {
+                            int64_t x = 0;
+                            if (a.a_col[g][f] >= 0) x = gf_fetch(a, w, a.a_col[g][f]).i;
+                            pr *= a.a_a[g][f] + a.a_b[g][f] * x;
+                        }
+                    }
+                    racc[g] += pr;
+                }
+                racc[VD_MAX_AGGS] += 1;
+            }
+            return;
+        }
+        if (__ballot_sync(VD_FULL, ok) == 0) return;  // nothing of this 32-row step qualifies
         int64_t key = 0;
         if (ok) {
             for (int k = 0; k < a.nkey && ok; ++k) {
@@ -1265,6 +1293,14 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
             }
         }
     }
+    if (SCALAR && warp < GF_CW) {
+#pragma unroll
+        for (int g = 0; g <= VD_MAX_AGGS; ++g) {
+            const int slot = g < NA ? g : (g == VD_MAX_AGGS ? NA : -1);
+            const int64_t t = warp_sum_i64(racc[g]);  // per-warp bound proven on the host
+            if (lane == 0 && slot >= 0) acc[(size_t)warp * NS + slot] = t;
+        }
+    }
     __syncthreads();
     // CTA fold of the warps' slots (int128), then the grid's (last CTA)
     for (int k = threadIdx.x; k < NS; k += GF_THREADS) {
@@ -1282,6 +1318,178 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
     if (!s_last) return;
     __threadfence();
     for (int k = threadIdx.x; k < NS; k += GF_THREADS) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
+            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[k], t);
+    }
+}
+
+// ============================================================================
+// FK grouped-fold fragment (Q9 shape): key = (dim[fk - bias] - subA) * mA +
+// (f(kb) - subB) * mB with f = calendar year (shared-memory table) or
+// identity, value = X * (a + b * Y) (32x32->64 IMAD.WIDE when proven narrow),
+// COUNT.  Base columns fk (i32), kb (i32), X, Y (i64) stream through the TMA
+// ring (24 B/row); the dimension column (u8) is gathered per row from L2.
+// Per-warp shared-memory group slots, filled by one leader lane per distinct
+// key of each 32-row step (__match_any_sync) -- the virtual scatter of
+// §3.1.3 at warp granularity.
+// ============================================================================
+constexpr int FKG_TILE = 2048;
+constexpr int FKG_CW = 16;  // consumer warps (latency hiding for the L2 gathers)
+constexpr int FKG_NT = FKG_CW * 32;
+constexpr int FKG_THREADS = FKG_NT + 32;
+
+struct FkgArgs {
+    const int32_t* fk;
+    const int32_t* kb;
+    const int64_t* x;
+    const int64_t* y;
+    const uint8_t* dim;
+    int64_t dim_len, bias;
+    int32_t subA, mA, subB, mB;
+    int32_t yfn, ylo, ydays;
+    int64_t a, b;
+    int32_t ngroups;
+    int32_t nstages;
+    int64_t n;
+    int32_t sum_slot, cnt_slot;  // plan aggregate indices (-1: absent)
+    int32_t naggs;
+};
+
+template <bool NARROW>
+__global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_constant__ FkgArgs a, int64_t ntiles,
+                                                            Slot16* __restrict__ parts, unsigned int* __restrict__ done,
+                                                            Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    constexpr int SB = FKG_TILE * (4 + 4 + 8 + 8);
+    int64_t* acc = reinterpret_cast<int64_t*>(smem + (size_t)a.nstages * SB);  // [FKG_CW][ngroups][2]
+    int64_t* sv = acc + (size_t)FKG_CW * a.ngroups * 2;                        // [FKG_CW][32]
+    int16_t* ytab = reinterpret_cast<int16_t*>(sv + FKG_CW * 32);
+    uint64_t* full = reinterpret_cast<uint64_t*>(ytab + ((a.ydays + 7) & ~7));
+    uint64_t* empty = full + a.nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < a.nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], FKG_CW);
+        }
+        fence_mbar_init();
+    }
+    for (int k = threadIdx.x; k < FKG_CW * a.ngroups * 2; k += FKG_THREADS) acc[k] = 0;
+    for (int k = threadIdx.x; k < a.ydays; k += FKG_THREADS) ytab[k] = (int16_t)year_of_day(a.ylo + k);
+    __syncthreads();
+    int64_t* wacc = acc + (size_t)warp * a.ngroups * 2;
+    int64_t* wsv = sv + warp * 32;
+
+    // one 32-row step of a warp: lane's row (fk, kb, x, y), valid flag
+    auto step = [&](bool valid, int32_t fk, int32_t kb, int64_t x, int64_t y) {
+        int key = -1;
+        int64_t v = 0;
+        if (valid) {
+            const int64_t p = (int64_t)fk - a.bias;
+            if (p >= 0 && p < a.dim_len && fk != INT32_MIN) {
+                const int d = __ldg(a.dim + p);
+                int kbv = kb;
+                if (a.yfn) {
+                    const int dd = kb - a.ylo;  // the table covers [min, max] of kb (metadata)
+                    kbv = (dd >= 0 && dd < a.ydays) ? (int)ytab[dd] : -0x40000000;
+                }
+                key = (d - a.subA) * a.mA + (kbv - a.subB) * a.mB;
+                if (d == 0xFF || kb == INT32_MIN || key < 0 || key >= a.ngroups) key = -1;
+                if (NARROW) {
+                    const int32_t f = (int32_t)a.a + (int32_t)a.b * (int32_t)y;
+                    v = (int64_t)(int32_t)x * (int64_t)f;
+                } else {
+                    v = x * (a.a + a.b * y);
+                }
+            }
+        }
+        wsv[lane] = v;
+        __syncwarp();
+        const unsigned m = __match_any_sync(VD_FULL, key);
+        if (key >= 0 && (__ffs(m) - 1) == lane) {
+            int64_t t = 0;
+            for (unsigned mm = m; mm; mm &= mm - 1) t += wsv[__ffs(mm) - 1];
+            wacc[2 * key] += t;
+            wacc[2 * key + 1] += __popc(m);
+        }
+        __syncwarp();
+    };
+
+    if (warp == FKG_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % a.nstages);
+                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * SB;
+                const int64_t r0 = tile * FKG_TILE;
+                mbar_expect_tx(&full[s], SB);
+                tma_load_1d(st, a.fk + r0, FKG_TILE * 4, &full[s], pol);
+                tma_load_1d(st + FKG_TILE * 4, a.kb + r0, FKG_TILE * 4, &full[s], pol);
+                tma_load_1d(st + FKG_TILE * 8, a.x + r0, FKG_TILE * 8, &full[s], pol);
+                tma_load_1d(st + FKG_TILE * 16, a.y + r0, FKG_TILE * 8, &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % a.nstages);
+            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            const uint8_t* st = smem + (size_t)s * SB;
+            constexpr int RPT = FKG_TILE / FKG_NT;
+            int32_t f[RPT], kb[RPT];
+            int64_t x[RPT], y[RPT];
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) {
+                const int r = threadIdx.x + k * FKG_NT;
+                f[k] = reinterpret_cast<const int32_t*>(st)[r];
+                kb[k] = reinterpret_cast<const int32_t*>(st + FKG_TILE * 4)[r];
+                x[k] = reinterpret_cast<const int64_t*>(st + FKG_TILE * 8)[r];
+                y[k] = reinterpret_cast<const int64_t*>(st + FKG_TILE * 16)[r];
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) step(true, f[k], kb[k], x[k], y[k]);
+        }
+        if (blockIdx.x == 0) {
+            for (int64_t base = ntiles * FKG_TILE + warp * 32; base < a.n; base += FKG_NT) {
+                const int64_t r = base + lane;
+                const bool ok = r < a.n;
+                step(ok, ok ? a.fk[r] : 0, ok ? a.kb[r] : 0, ok ? a.x[r] : 0, ok ? a.y[r] : 0);
+            }
+        }
+    }
+    __syncthreads();
+    const int NS = a.ngroups * (a.naggs + 1);
+    // CTA fold (int128) into [ngroups][naggs+1] directly in the plan's layout
+    for (int k = threadIdx.x; k < NS; k += FKG_THREADS) {
+        const int g = k / (a.naggs + 1), ag = k % (a.naggs + 1);
+        const int src = (ag == a.naggs || ag == a.cnt_slot) ? 1 : 0;
+        i128 t = 0;
+        for (int w = 0; w < FKG_CW; ++w) t += (i128)acc[((size_t)w * a.ngroups + g) * 2 + src];
+        put_i128(&parts[(size_t)blockIdx.x * NS + k], t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    for (int k = threadIdx.x; k < NS; k += FKG_THREADS) {
         i128 t = 0;
         for (unsigned b = 0; b < gridDim.x; ++b) {
             Slot16 x;
@@ -1888,6 +2096,104 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
     return VD_OK;
 }
 
+// ---- FK grouped-fold (Q9 shape) matching ---------------------------------------------
+static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                         void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    const char* var = getenv("VD_FKG_VARIANT");
+    if (var && strcmp(var, "off") == 0) return VD_OK;
+    if (p->pred.nconj != 0 || p->ngathers != 1 || p->nkeyparts != 2 || p->ngroups > 512) return VD_OK;
+    const vd_gatherspec& gs = p->gathers[0];
+    const vd_column& dim = dims[gs.dim_col];
+    if (cols[gs.fk_col].dtype != VD_I32 || dim.dtype != VD_U8) return VD_OK;
+    // key part A: the gathered column (identity); key part B: a base i32 column
+    int ia = -1, ib = -1;
+    for (int k = 0; k < 2; ++k) {
+        if (p->key[k].col == ncols && p->key[k].fn == 0) ia = k;
+        else if (p->key[k].col < ncols && cols[p->key[k].col].dtype == VD_I32) ib = k;
+    }
+    if (ia < 0 || ib < 0) return VD_OK;
+    // aggregates: one SUM(X * (a + b*Y)) over i64 base columns, COUNT
+    FkgArgs A;
+    std::memset(&A, 0, sizeof(A));
+    A.sum_slot = A.cnt_slot = -1;
+    A.naggs = p->naggs;
+    int X = -1, Y = -1;
+    for (int g = 0; g < p->naggs; ++g) {
+        const vd_agg& ag = p->aggs[g];
+        if (ag.kind == VD_AGG_COUNT) { if (A.cnt_slot >= 0) return VD_OK; A.cnt_slot = g; continue; }
+        if (ag.kind != VD_AGG_SUM || A.sum_slot >= 0 || ag.nfactors != 2 || !plain_col(ag.f[0])) return VD_OK;
+        X = ag.f[0].col;
+        Y = ag.f[1].col;
+        if (X >= ncols || Y < 0 || Y >= ncols || cols[X].dtype != VD_I64 || cols[Y].dtype != VD_I64) return VD_OK;
+        A.a = ag.f[1].a;
+        A.b = ag.f[1].b;
+        A.sum_slot = g;
+    }
+    if (A.sum_slot < 0) return VD_OK;
+    const int kbcol = p->key[ib].col, fkcol = gs.fk_col;
+    for (int c : {fkcol, kbcol, X, Y})
+        if (((uintptr_t)cols[c].data % 16) != 0) return VD_OK;
+    // exactness: |X*(a+bY)| * rows per warp < 2^63; narrow if everything fits 32 bits
+    Bound bx = col_bound(p, cols, ncols, dims, X), by = col_bound(p, cols, ncols, dims, Y);
+    if (!bx.known || !by.known) return VD_OK;
+    vd_factor fy;
+    fy.col = Y; fy.a = A.a; fy.b = A.b;
+    const double fmx = factor_absmax(fy, by), xmx = std::max(std::fabs(bx.lo), std::fabs(bx.hi));
+    const int grid = num_sms();
+    const double rows_per_warp = std::ceil((double)n / ((double)grid * FKG_CW)) + FKG_TILE;
+    if (xmx * fmx * rows_per_warp >= 9.0e18) return VD_OK;
+    const bool narrow = xmx < 2147483647.0 && fmx < 2147483647.0 && xmx * fmx < 9.0e18 &&
+                        std::max(std::fabs(by.lo), std::fabs(by.hi)) < 2147483647.0 && std::fabs((double)A.a) < 2.0e9 &&
+                        std::fabs((double)A.b) < 2.0e9;
+    A.fk = (const int32_t*)cols[fkcol].data;
+    A.kb = (const int32_t*)cols[kbcol].data;
+    A.x = (const int64_t*)cols[X].data;
+    A.y = (const int64_t*)cols[Y].data;
+    A.dim = (const uint8_t*)dim.data;
+    A.dim_len = dim.len;
+    A.bias = gs.bias;
+    A.subA = (int32_t)p->key[ia].sub;
+    A.mA = (int32_t)p->key[ia].mult;
+    A.subB = (int32_t)p->key[ib].sub;
+    A.mB = (int32_t)p->key[ib].mult;
+    A.yfn = p->key[ib].fn;
+    A.ylo = 0;
+    A.ydays = 0;
+    if (A.yfn) {
+        if (!(cols[kbcol].has_minmax && cols[kbcol].max - cols[kbcol].min < GF_MAXYEARDAYS)) return VD_OK;
+        A.ylo = (int32_t)cols[kbcol].min;
+        A.ydays = (int32_t)(cols[kbcol].max - cols[kbcol].min + 1);
+    }
+    A.ngroups = (int32_t)p->ngroups;
+    A.n = n;
+    constexpr size_t SB = FKG_TILE * 24;
+    const size_t fixed = (size_t)FKG_CW * p->ngroups * 16 + FKG_CW * 32 * 8 + (size_t)((A.ydays + 7) & ~7) * 2 +
+                         2 * GF_MAXSTAGES * 8;
+    const size_t budget = 200 * 1024;
+    if (fixed + 2 * SB > budget) return VD_OK;
+    int ns = (int)((budget - fixed) / SB);
+    A.nstages = ns > GF_MAXSTAGES ? GF_MAXSTAGES : ns;
+    const size_t smem = fixed + (size_t)A.nstages * SB;
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    if (narrow) {
+        cudaFuncSetAttribute(k_pipe_fkg<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_fkg<true><<<grid, FKG_THREADS, smem, s>>>(A, n / FKG_TILE, parts, dn, (Slot16*)out);
+    } else {
+        cudaFuncSetAttribute(k_pipe_fkg<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_fkg<false><<<grid, FKG_THREADS, smem, s>>>(A, n / FKG_TILE, parts, dn, (Slot16*)out);
+    }
+    ++*nl;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    set_fragment("fk_group");
+    *done = true;
+    return VD_OK;
+}
+
 // ---- gather-fold matching -------------------------------------------------------
 static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
                         void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
@@ -1923,17 +2229,66 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         A.g_len[g] = d.len;
         A.g_dt[g] = d.dtype;
     }
-    // predicate, base terms first within each conjunction
+    // predicate: hoist base-column terms shared by every conjunction (AND
+    // distributes over OR), then per conjunction base terms first (no gather
+    // for a row that already failed), equality / IN terms (usually the most
+    // selective) before ranges
     vd_pred pr = p->pred;
+    auto same = [](const vd_term& x, const vd_term& y) {
+        return x.col == y.col && x.cmp == y.cmp && x.ival == y.ival && x.fval == y.fval;
+    };
+    A.ncommon = 0;
+    if (pr.nconj >= 1) {
+        vd_conj& c0 = pr.conj[0];
+        for (int t = 0; t < c0.nterms; ++t) {
+            const vd_term& cand = c0.terms[t];
+            if (cand.col >= ncols) continue;
+            bool everywhere = true;
+            for (int c = 1; c < pr.nconj && everywhere; ++c) {
+                bool found = false;
+                for (int u = 0; u < pr.conj[c].nterms; ++u) found = found || same(cand, pr.conj[c].terms[u]);
+                everywhere = found;
+            }
+            if (!everywhere) continue;
+            bool dup = false;
+            for (int k = 0; k < A.ncommon; ++k)
+                dup = dup || (A.common[k].col == cand.col && A.common[k].cmp == cand.cmp && A.common[k].iv == cand.ival &&
+                              A.common[k].fv == cand.fval);
+            if (!dup && A.ncommon < VD_MAX_TERMS) {
+                A.common[A.ncommon].col = cand.col;
+                A.common[A.ncommon].cmp = cand.cmp;
+                A.common[A.ncommon].iv = cand.ival;
+                A.common[A.ncommon].fv = cand.fval;
+                ++A.ncommon;
+            }
+        }
+    }
+    auto rank = [&](const vd_term& t) {
+        const bool base = t.col < ncols;
+        const bool eq = t.cmp == VD_CMP_EQ || t.cmp == VD_CMP_IN;
+        return (base ? 0 : 2) + (eq ? 0 : 1);
+    };
+    bool always = false;  // a conjunction reduced to the common terms only
     for (int c = 0; c < pr.nconj; ++c) {
         vd_conj& cj = pr.conj[c];
         vd_term tmp[VD_MAX_TERMS];
         int k = 0;
-        for (int t = 0; t < cj.nterms; ++t) if (cj.terms[t].col < ncols) tmp[k++] = cj.terms[t];
-        A.nbase[c] = k;
-        for (int t = 0; t < cj.nterms; ++t) if (cj.terms[t].col >= ncols) tmp[k++] = cj.terms[t];
-        for (int t = 0; t < cj.nterms; ++t) cj.terms[t] = tmp[t];
+        for (int r = 0; r < 4; ++r)
+            for (int t = 0; t < cj.nterms; ++t) {
+                bool hoisted = false;
+                for (int h = 0; h < A.ncommon; ++h)
+                    hoisted = hoisted || (A.common[h].col == cj.terms[t].col && A.common[h].cmp == cj.terms[t].cmp &&
+                                          A.common[h].iv == cj.terms[t].ival && A.common[h].fv == cj.terms[t].fval);
+                if (!hoisted && rank(cj.terms[t]) == r) tmp[k++] = cj.terms[t];
+            }
+        int nb = 0;
+        for (int t = 0; t < k; ++t) nb += tmp[t].col < ncols;
+        A.nbase[c] = nb;
+        cj.nterms = k;
+        for (int t = 0; t < k; ++t) cj.terms[t] = tmp[t];
+        if (k == 0) always = true;
     }
+    if (always) pr.nconj = 0;  // the common terms decide
     make_devpred(&pr, &A.pred);
     // key
     A.nkey = p->nkeyparts;
@@ -1992,13 +2347,16 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     const int mode = p->sel_mode == VD_SEL_PREDICATED ? 1 : 0;
+#define GF_LAUNCH(M, SC)                                                                              \
+    cudaFuncSetAttribute(k_pipe_gf<M, SC>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);    \
+    k_pipe_gf<M, SC><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
+    const bool scalar = p->ngroups == 1;
     if (mode) {
-        cudaFuncSetAttribute(k_pipe_gf<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_gf<1><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
+        if (scalar) { GF_LAUNCH(1, true) } else { GF_LAUNCH(1, false) }
     } else {
-        cudaFuncSetAttribute(k_pipe_gf<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_gf<0><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
+        if (scalar) { GF_LAUNCH(0, true) } else { GF_LAUNCH(0, false) }
     }
+#undef GF_LAUNCH
     ++*nl;
     e = cudaGetLastError();
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
@@ -2116,6 +2474,8 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         vd_status st = try_q1(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+        st = try_fkg(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;

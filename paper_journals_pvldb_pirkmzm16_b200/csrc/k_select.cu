@@ -19,8 +19,11 @@
 //                        the next step.  The valid prefix is then streamed
 //                        out with coalesced stores.  No lane of one store
 //                        instruction shares an address with another.
+#include <algorithm>
+#include <cmath>
 #include <cstdlib>
 #include <cstring>
+#include <type_traits>
 
 #include "vd_common.cuh"
 #include "vd_internal.h"
@@ -93,7 +96,13 @@ struct TermFlags {
     int cmp;
     int64_t iv;
     double fv;
+    // interval form lo <= x <= hi of the term (ivl != 0), with epsilon
+    // excluded by the bounds (int: lo > MIN / u8: hi < 0xFF; float: NaN
+    // fails every comparison); computed on the host
+    int ivl;
+    T lo, hi;
     __device__ __forceinline__ bool test(T x) const {
+        if (ivl) return x >= lo && x <= hi;
         if (Eps<T>::is(x)) return false;
         if (IsFloat<T>::value) return cmp_flt(cmp, (double)x, fv);
         return cmp_int(cmp, (int64_t)x, iv);
@@ -307,23 +316,31 @@ __global__ void __launch_bounds__(SEL_THREADS) k_select(F fl, int64_t n, int32_t
 constexpr int BM_THREADS = 256;
 constexpr int BM_CHUNK = 1024;  // rows per warp chunk = 32 words
 
-// Bitmap layout ("ballot order"): chunk c holds rows c*1024 + q*128 + 4*L + j
-// (q = 0..7, lane L = 0..31, j = 0..3) as bit L of word c*32 + q*4 + j, so
-// every load instruction of the flag pass reads 512 contiguous bytes and
-// every word is one warp ballot.
+// Bitmap layout: chunk c, word w (0..31), bit i <-> row c*1024 + 32*w + i.
+// Flag pass: each load instruction reads 512 contiguous bytes (lane L takes
+// rows q*128 + 4L .. 4L+3), the warp ballots each of the 4 row phases, and
+// lane w assembles word w from the four ballots of its 128-row block by
+// spreading bytes (word = interleave of 4 ballot bytes).
+__device__ __forceinline__ uint32_t spread8(uint32_t x) {  // bit k -> bit 4k
+    x = (x | (x << 12)) & 0x000F000Fu;
+    x = (x | (x << 6)) & 0x03030303u;
+    x = (x | (x << 3)) & 0x11111111u;
+    return x;
+}
+
 template <typename T, bool ALIGNED>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNED> fl, int64_t n,
                                                              uint32_t* __restrict__ bits,
                                                              int32_t* __restrict__ counts, int64_t nchunks) {
-    const int lane = threadIdx.x & 31;
+    __shared__ uint32_t s_bal[BM_THREADS / 32][32];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
+    uint32_t* bal = s_bal[warp];
     for (int64_t c = gw; c < nchunks; c += nw) {
         typename TermFlags<T, ALIGNED>::Raw raw[8];
 #pragma unroll
         for (int q = 0; q < 8; ++q) fl.load(c * BM_CHUNK + q * 128 + lane * 4, n, raw[q]);
-        uint32_t mine = 0;
-        int cnt = 0;
 #pragma unroll
         for (int q = 0; q < 8; ++q) {
             bool f[4];
@@ -331,16 +348,25 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNE
 #pragma unroll
             for (int j = 0; j < 4; ++j) {
                 const uint32_t b = __ballot_sync(VD_FULL, f[j]);
-                cnt += __popc(b);
-                if (lane == q * 4 + j) mine = b;
+                if (lane == 0) bal[q * 4 + j] = b;  // bit L <-> row q*128 + 4L + j
             }
         }
-        bits[c * 32 + lane] = mine;
+        __syncwarp();
+        // word w = rows 32w..32w+31 = q-block w/4, lanes 8(w%4) .. 8(w%4)+7
+        const int q = lane >> 2, m = lane & 3;
+        uint32_t word = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) word |= spread8((bal[q * 4 + j] >> (8 * m)) & 0xFFu) << j;
+        __syncwarp();
+        bits[c * 32 + lane] = word;
+        int cnt = __popc(word);
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) cnt += __shfl_xor_sync(VD_FULL, cnt, o);
         if (lane == 0) counts[c] = cnt;
     }
 }
 
-// Per-row predicates (several columns, run heads), same layout.
+// Per-row predicates (several columns, run heads): ballot j is word j.
 template <class F>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_bal(F fl, int64_t n, uint32_t* __restrict__ bits,
                                                              int32_t* __restrict__ counts, int64_t nchunks) {
@@ -349,17 +375,15 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_bal(F fl, int64_t n, ui
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
     for (int64_t c = gw; c < nchunks; c += nw) {
         uint32_t mine = 0;
-        int cnt = 0;
-#pragma unroll 2
-        for (int q = 0; q < 8; ++q) {
-#pragma unroll
-            for (int j = 0; j < 4; ++j) {
-                const uint32_t b = __ballot_sync(VD_FULL, fl.eval1(c * BM_CHUNK + q * 128 + lane * 4 + j, n));
-                cnt += __popc(b);
-                if (lane == q * 4 + j) mine = b;
-            }
+#pragma unroll 4
+        for (int j = 0; j < 32; ++j) {
+            const uint32_t b = __ballot_sync(VD_FULL, fl.eval1(c * BM_CHUNK + j * 32 + lane, n));
+            if (lane == j) mine = b;
         }
         bits[c * 32 + lane] = mine;
+        int cnt = __popc(mine);
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) cnt += __shfl_xor_sync(VD_FULL, cnt, o);
         if (lane == 0) counts[c] = cnt;
     }
 }
@@ -369,55 +393,58 @@ __global__ void k_sel_total(const int64_t* __restrict__ offs, const int32_t* __r
     *out_count = nchunks > 0 ? offs[nchunks - 1] + counts[nchunks - 1] : 0;
 }
 
+// Position pass: lane w owns word w (rows 32w..32w+31 of the chunk); the
+// chunk's positions are assembled in a shared-memory stage and stream out
+// with coalesced stores.
+//   branching : only the qualifying rows are written to the stage;
+//   predicated: cursor arithmetic -- every row is written, qualifying rows
+//               at the lane's cursor and the others past the chunk's count.
 template <int MODE>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __restrict__ bits,
                                                           const int64_t* __restrict__ offs, int64_t nchunks,
                                                           int32_t* __restrict__ out) {
-    __shared__ int32_t s_stage[MODE == 1 ? (BM_THREADS / 32) * 128 : 1];
+    // stage index k is stored at k + k/32 (one pad word per 32): lanes whose
+    // cursors are 32 apart hit different banks
+    __shared__ int32_t s_stage[(BM_THREADS / 32) * (BM_CHUNK + BM_CHUNK / 32)];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const unsigned lt = lanemask_lt();
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
+    int32_t* st = s_stage + warp * (BM_CHUNK + BM_CHUNK / 32);
     for (int64_t c = gw; c < nchunks; c += nw) {
-        const uint32_t myword = bits[c * 32 + lane];
-        int64_t base = offs[c];
-        for (int q = 0; q < 8; ++q) {
-            uint32_t b[4];
-            int cnt = 0, before = 0, mine = 0;
+        const uint32_t w = bits[c * 32 + lane];
+        const int pc = __popc(w);
+        int incl = pc;
 #pragma unroll
-            for (int j = 0; j < 4; ++j) {
-                b[j] = __shfl_sync(VD_FULL, myword, q * 4 + j);
-                cnt += __popc(b[j]);
-                before += __popc(b[j] & lt);
-                mine += (b[j] >> lane) & 1u;
-            }
-            const int32_t row = (int32_t)(c * BM_CHUNK + q * 128 + lane * 4);
-            if (MODE == 0) {
-                // branching: a qualifying row stores its position (lanes of a
-                // store instruction write increasing, nearly contiguous slots)
-                int k = before;
-#pragma unroll
-                for (int j = 0; j < 4; ++j)
-                    if ((b[j] >> lane) & 1u) out[base + k++] = row + j;
-            } else {
-                // predicated (cursor arithmetic): every row of the 128-row block
-                // is written; qualifying rows at the cursor, the others past it
-                int32_t* st = s_stage + warp * 128;
-                int sel = before, unsel = cnt + (lane * 4 - before);
-#pragma unroll
-                for (int j = 0; j < 4; ++j) {
-                    const int f = (b[j] >> lane) & 1u;
-                    st[f ? sel : unsel] = row + j;
-                    sel += f;
-                    unsel += 1 - f;
-                }
-                __syncwarp();
-                for (int k = lane; k < cnt; k += 32) out[base + k] = st[k];
-                __syncwarp();
-            }
-            (void)mine;
-            base += cnt;
+        for (int o = 1; o < 32; o <<= 1) {
+            const int u = __shfl_up_sync(VD_FULL, incl, o);
+            if (lane >= o) incl += u;
         }
+        const int excl = incl - pc;
+        const int total = __shfl_sync(VD_FULL, incl, 31);
+        const int32_t row0 = (int32_t)(c * BM_CHUNK + lane * 32);
+        if (MODE == 0) {
+            uint32_t m = w;
+            int k = excl;
+            while (m) {
+                st[k + (k >> 5)] = row0 + (__ffs(m) - 1);
+                ++k;
+                m &= m - 1;
+            }
+        } else {
+            int sel = excl, unsel = total + (lane * 32 - excl);
+#pragma unroll
+            for (int i = 0; i < 32; ++i) {
+                const int f = (w >> i) & 1u;
+                const int k = f ? sel : unsel;
+                st[k + (k >> 5)] = row0 + i;
+                sel += f;
+                unsel += 1 - f;
+            }
+        }
+        __syncwarp();
+        const int64_t base = offs[c];
+        for (int k = lane; k < total; k += 32) out[base + k] = st[k + (k >> 5)];
+        __syncwarp();
     }
 }
 
@@ -502,13 +529,56 @@ static cudaError_t run_select(const F& fl, int64_t n, int32_t* out_pos, int64_t*
     return cudaGetLastError();
 }
 
+// Interval form [lo, hi] of one comparison on a column of T (epsilon
+// excluded); false for NE / IN.
+template <typename T>
+static bool term_interval_t(const DevTerm& t, T* lo, T* hi) {
+    if (IsFloat<T>::value) {
+        // exact for f32 / f64 values against a double constant
+        const double c = t.fv;
+        double l = -HUGE_VAL, h = HUGE_VAL;
+        auto down = [](double x) { T f = (T)x; if ((double)f > x) f = nextafter(f, (T)-HUGE_VAL); return f; };
+        auto up = [](double x) { T f = (T)x; if ((double)f < x) f = nextafter(f, (T)HUGE_VAL); return f; };
+        switch (t.cmp) {
+        case VD_CMP_GT: l = (double)nextafter(down(c), (T)HUGE_VAL); break;
+        case VD_CMP_GE: l = (double)up(c); break;
+        case VD_CMP_LT: h = (double)nextafter(up(c), (T)-HUGE_VAL); break;
+        case VD_CMP_LE: h = (double)down(c); break;
+        case VD_CMP_EQ: if ((double)(T)c != c) { l = 1; h = 0; } else { l = h = c; } break;
+        default: return false;
+        }
+        *lo = (T)l;
+        *hi = (T)h;
+        return true;
+    }
+    const int64_t tmin = std::is_same<T, uint8_t>::value ? 0 : (std::is_same<T, int32_t>::value ? INT32_MIN + 1 : INT64_MIN + 1);
+    const int64_t tmax = std::is_same<T, uint8_t>::value ? 0xFE : (std::is_same<T, int32_t>::value ? INT32_MAX : INT64_MAX);
+    int64_t l = tmin, h = tmax;
+    const int64_t c = t.iv;
+    switch (t.cmp) {
+    case VD_CMP_GT: if (c >= tmax) { l = 1; h = 0; } else l = std::max(l, c + 1); break;
+    case VD_CMP_GE: l = std::max(l, c); break;
+    case VD_CMP_LT: if (c <= tmin) { l = 1; h = 0; } else h = std::min(h, c - 1); break;
+    case VD_CMP_LE: h = std::min(h, c); break;
+    case VD_CMP_EQ: l = std::max(l, c); h = std::min(h, c); break;
+    default: return false;
+    }
+    if (l > h) { l = 1; h = 0; }
+    if (std::is_same<T, uint8_t>::value && l > h) { *lo = (T)1; *hi = (T)0; return true; }
+    *lo = (T)l;
+    *hi = (T)h;
+    return true;
+}
+
 template <int MODE, typename T>
 static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int32_t* out_pos, int64_t* out_count,
                                  void* ws, cudaStream_t s, int* nl) {
     size_t vecbytes = sizeof(T) * 4 > 16 ? 16 : sizeof(T) * 4;
     bool aligned = ((uintptr_t)p % vecbytes) == 0;
+    T ilo = T(0), ihi = T(0);
+    const int ivl = term_interval_t<T>(t, &ilo, &ihi) ? 1 : 0;
     if (aligned) {
-        TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv};
+        TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L, int grid) {
@@ -516,7 +586,7 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
             },
             n, out_pos, out_count, ws, s, nl);
     }
-    TermFlags<T, false> f{(const T*)p, t.cmp, t.iv, t.fv};
+    TermFlags<T, false> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
     if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
     return run_select_bitmap<MODE>(
         [&](const BmLayout& L, int grid) {

@@ -167,7 +167,7 @@ def test_fkj_q9_vs_oracle(sel_mode, generic, n):
     dkeep, dviews = load([supp[c] for c in plans.Q9_DIMS])
     plan = plans.q9(sel_mode, force_generic=generic)
     got = vd.decode_partials(run(plan, views, len(li["l_suppkey"]), dviews,
-                                 want=("generic",) if generic else ("gather_fold",))[0], plan)
+                                 want=("generic",) if generic else ("fk_group",))[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
@@ -242,3 +242,23 @@ def test_selective_sum_f32_interval_edges(op, c):
     assert got[0][1] == int(m.sum())
     ref = float(np.sum(x[m]))
     assert got[0][0] == ref or abs(got[0][0] - ref) <= 1e-9 * abs(ref)
+
+
+@pytest.mark.parametrize("variant", ["gather_fold", "generic"])
+def test_fkj_q9_gather_fold_fragment(variant):
+    """The Q9 plan through the general gather-fold fragment (the FK grouped
+    fragment disabled) and through the generic one."""
+    import os
+    sf = 0.05
+    li = lineitem(sf, 200003)
+    part, supp = _dims(sf)
+    exp = oracle.fkj(1, li, part, supp)
+    keep, views = load([li[c] for c in plans.Q9_COLS])
+    dkeep, dviews = load([supp[c] for c in plans.Q9_DIMS])
+    plan = plans.q9(force_generic=(variant == "generic"))
+    os.environ["VD_FKG_VARIANT"] = "off"
+    try:
+        got = vd.decode_partials(run(plan, views, len(li["l_suppkey"]), dviews, want=(variant,))[0], plan)
+    finally:
+        del os.environ["VD_FKG_VARIANT"]
+    assert {k: tuple(v[:2]) for k, v in got.items()} == exp
