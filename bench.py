@@ -35,7 +35,7 @@ METRIC = "rows/s and achieved HBM GB/s (% of peak) for TPC-H Q1/Q6 at 1/2/4/8 B2
 # Algorithmic bytes per row: every
 # column each query reads, once.
 BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "q19": 4 + 3 * 8 + 1 + 1,
-                 "q9": 4 + 4 + 2 * 8}
+                 "q9": 4 + 4 + 2 * 8, "fkjsel": 4 + 4}
 
 
 def parse():
@@ -44,9 +44,12 @@ def parse():
     ap.add_argument("--steps", type=int, default=None)
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
-    ap.add_argument("--workload", default="q1", choices=["q1", "q6", "select", "selpos", "q19", "q9"])
+    ap.add_argument("--workload", default="q1",
+                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused"])
+    ap.add_argument("--chunk", type=int, default=0,
+                    help="select_unfused: rows per materialised chunk (0 = whole table; Fig 15 'Vectorized')")
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
-    ap.add_argument("--sel-mode", default="branch", choices=["branch", "predicated"])
+    ap.add_argument("--sel-mode", default="branch", choices=["branch", "predicated", "lookup"])
     ap.add_argument("--selectivity", type=float, default=0.5, help="select workload: fraction selected")
     ap.add_argument("--rows", type=int, default=None, help="select workload: rows (default 1e9)")
     ap.add_argument("--generic", action="store_true", help="force the generic fragment")
@@ -60,7 +63,7 @@ def parse():
 
 
 def default_sf(w):
-    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0}[w]
+    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0}[w]
 
 
 # ---------------------------------------------------------------------------
@@ -201,6 +204,8 @@ def main():
         return reference_arm(args, rank, world, sf)
     if args.workload == "selpos":
         return selpos_main(args, rank, world, local)
+    if args.workload == "select_unfused":
+        return unfused_main(args, rank, world, local)
 
     import torch
     import torch.distributed as dist
@@ -217,11 +222,14 @@ def main():
     w = args.workload
     if w == "select":
         n_total = args.rows or 10**9
+    elif w == "fkjsel":
+        n_total = args.rows or 200_000_000
     else:
         n_total = gen.lineitem_rows(sf)
     a, b = rank * n_total // world, (rank + 1) * n_total // world
     n = b - a
-    sel_mode = vd.VD_SEL_PREDICATED if args.sel_mode == "predicated" else vd.VD_SEL_BRANCH
+    sel_mode = {"branch": vd.VD_SEL_BRANCH, "predicated": vd.VD_SEL_PREDICATED,
+                "lookup": vd.VD_SEL_PREDICATED_LOOKUP}[args.sel_mode]
 
     # ---- a1: columns generated in HBM (row range [a, b)), min/max via vd folds
     def make(col, length, row0, sfv=sf, **kw):
@@ -257,11 +265,30 @@ def main():
         names, plan = plans.Q9_COLS, plans.q9(sel_mode, force_generic=args.generic)
         for d in plans.Q9_DIMS:
             dims.append(make(gen.SUPPLIER_COLS[d], gen.supplier_rows(sf), 0))
+    elif w == "fkjsel":
+        # Fig 16: fact(fk, v) x target(v) through fk - 1, v < threshold, sum(target.v)
+        m = plans.FKJSEL_TARGET_ROWS
+        names = ["fk", "v"]
+        thr = int(round(args.selectivity * plans.FKJSEL_VMAX))
+        plan = plans.fkjsel(thr, sel_mode, force_generic=args.generic)
+        t = torch.empty(m, dtype=torch.int64, device=dev)
+        gen.device(gen.I64_UNIFORM, t.data_ptr(), m, 0, seed=args.seed + 2, p0=0, p1=10**6, stream=stream.cuda_stream)
+        dims.append(t)
     else:
         names = ["v"]
         plan = plans.selsum(float(__import__("numpy").float32(args.selectivity)), sel_mode,
                             force_generic=args.generic)
     for nm in names:
+        if w == "fkjsel":
+            c = torch.empty(n, dtype=torch.int32, device=dev)
+            if nm == "fk":
+                gen.device(gen.I32_UNIFORM, c.data_ptr(), n, a, seed=args.seed, p0=1, p1=plans.FKJSEL_TARGET_ROWS,
+                           stream=stream.cuda_stream)
+            else:
+                gen.device(gen.I32_UNIFORM, c.data_ptr(), n, a, seed=args.seed + 1, p0=0, p1=plans.FKJSEL_VMAX - 1,
+                           stream=stream.cuda_stream)
+            cols.append(c)
+            continue
         col = gen.F32_UNIFORM if nm == "v" else gen.LINEITEM_COLS[nm]
         cols.append(make(col, n, a))
     torch.cuda.synchronize()
@@ -343,7 +370,8 @@ def main():
         "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
         "config": {
             "workload": {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
-                         "q9": f"fkj_q9_sf{sf:g}", "select": f"select_f32_{n_total}_s{args.selectivity:g}"}[w],
+                         "q9": f"fkj_q9_sf{sf:g}", "select": f"select_f32_{n_total}_s{args.selectivity:g}",
+                         "fkjsel": f"fkjsel_{n_total}x{plans.FKJSEL_TARGET_ROWS}_s{args.selectivity:g}"}[w],
             "rows": n_total, "rows_per_gpu": n, "sf": sf, "sel_mode": args.sel_mode,
             "fragment": "generic" if args.generic else "specialised",
             "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
@@ -481,6 +509,79 @@ class Comm:
         if self.world > 1:
             self.dist.barrier()
             self.dist.destroy_process_group()
+
+
+def unfused_main(args, rank, world, local):
+    """Selective aggregation without fusion (Fig 15's Materialize / Break, and
+    with --chunk its 'Vectorized' cache-sized chunks): per chunk
+    select -> int32 positions (materialised), gather the values (materialised),
+    FoldSum the chunk (positions past the count are -1 = epsilon, skipped by the
+    fold), then FoldSum the chunk partials.  Compare with --workload select."""
+    import numpy as np
+    import torch
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % ndev)
+    dev = torch.device("cuda", local % ndev)
+    comm = Comm(world, args.dist_backend, dev)
+    stream = torch.cuda.current_stream()
+    n_total = args.rows or 10**9
+    a, b = rank * n_total // world, (rank + 1) * n_total // world
+    n = b - a
+    v = torch.empty(n, dtype=torch.float32, device=dev)
+    gen.device(gen.F32_UNIFORM, v.data_ptr(), n, a, seed=args.seed, stream=stream.cuda_stream)
+    C = args.chunk if args.chunk > 0 else n
+    nch = (n + C - 1) // C
+    t = float(np.float32(args.selectivity))
+    p = vd.pred([[(0, "<", t)]])
+    fn = vd.select_predicated if args.sel_mode == "predicated" else vd.select_branch
+    pos = torch.empty(C, dtype=torch.int32, device=dev)
+    vals = torch.empty(C, dtype=torch.float32, device=dev)
+    cnt = torch.zeros(1, dtype=torch.int64, device=dev)
+    parts = torch.zeros(nch, dtype=torch.float64, device=dev)
+    total = torch.zeros(1, dtype=torch.float64, device=dev)
+    ws = vd.alloc_ws(max(vd.workspace_bytes(vd.VD_OP_SELECT, C), vd.workspace_bytes(vd.VD_OP_FOLD, C)), dev)
+    views = [vd.column(v[k * C:min(n, (k + 1) * C)]) for k in range(nch)]
+
+    def step():
+        for k in range(nch):
+            m = views[k].len
+            pos.fill_(-1)  # materialised buffer, epsilon beyond the count
+            fn([views[k]], m, p, out_pos=pos, out_count=cnt, ws=ws, stream=stream)
+            vd.gather(views[k], pos, m, 0, vals, stream=stream)
+            pv = parts[k:k + 1]
+            vd.fold_sum(vd.column(vals, length=m), None, out=pv, ws=ws, stream=stream)
+        vd.fold_sum(vd.column(parts), None, out=total, ws=ws, stream=stream)
+
+    for _ in range(max(args.warmup, 3)):
+        step()
+    torch.cuda.synchronize()
+    steps = args.steps or 20
+    comm.barrier()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    ms = comm.max([e0.elapsed_time(e1) / steps])[0]
+    peak, kind = hbm_peak()
+    alg = 4 * n / (ms * 1e-3) / 1e9
+    line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "f32/f64", "data": "synthetic (f32 U[0,1))",
+            "config": {"workload": f"select_unfused_{n_total}_s{args.selectivity:g}_chunk{C}",
+                       "sel_mode": args.sel_mode, "chunks": nch},
+            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
+                         "peak_kind": kind, "traffic": None, "kernel": "select+gather+fold (unfused)",
+                         "kernel_ms": ms},
+            "result": float(total.item()), "e2e": None}
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    comm.close()
 
 
 def _dt(col):

@@ -133,8 +133,15 @@ typedef struct {
  *   PREDICATED : branch-free cursor arithmetic -- every row is written at the
  *                output cursor and the cursor advances by the predicate
  *                (selection); every row is loaded and its contribution is
- *                multiplied by the 0/1 predicate (aggregation). */
-typedef enum { VD_SEL_BRANCH = 0, VD_SEL_PREDICATED = 1 } vd_sel_mode;
+ *                multiplied by the 0/1 predicate (aggregation: "Predicated
+ *                Aggregation" of Fig 16);
+ *   PREDICATED_LOOKUP : (pipelines with gathers) the FK position is
+ *                multiplied by the predicate before the lookup, so rows that
+ *                do not qualify all read position 0 -- one "very hot" cache
+ *                line -- and their contribution is still multiplied by the
+ *                predicate ("Predicated Lookups").
+ * All modes return identical results. */
+typedef enum { VD_SEL_BRANCH = 0, VD_SEL_PREDICATED = 1, VD_SEL_PREDICATED_LOOKUP = 2 } vd_sel_mode;
 
 /* ---------------------------------------------------------------------- */
 /* Misc                                                                    */

@@ -1116,17 +1116,22 @@ __device__ __forceinline__ Val gf_base(const GfArgs& a, const GfRow& w, int c) {
     return fetch_typed(a.col[c], a.dt[c], w.g);
 }
 
-__device__ __forceinline__ Val gf_fetch(const GfArgs& a, const GfRow& w, int c) {
+// zero_pos: predicated lookups (Fig 16) -- the position is multiplied by the
+// 0/1 predicate, so a non-qualifying row reads slot 0.
+__device__ __forceinline__ Val gf_fetch(const GfArgs& a, const GfRow& w, int c, bool zero_pos = false) {
     if (c < a.ncols) return gf_base(a, w, c);
     const int g = c - a.ncols;
-    Val fk = gf_base(a, w, a.g_fk[g]);
     Val out;
     out.eps = true;
     out.isf = false;
     out.i = 0;
     out.f = 0;
-    if (fk.eps) return out;
-    const int64_t p = fk.i - a.g_bias[g];
+    int64_t p = 0;
+    if (!zero_pos) {
+        Val fk = gf_base(a, w, a.g_fk[g]);
+        if (fk.eps) return out;
+        p = fk.i - a.g_bias[g];
+    }
     if (p < 0 || p >= a.g_len[g]) return out;
     return fetch_typed(a.g_p[g], a.g_dt[g], p);
 }
@@ -1187,21 +1192,31 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
     auto process = [&](const GfRow& w, bool valid) {
         bool ok = valid && gf_pred(a, w);
         if (SCALAR) {
-            if (ok) {
+            // MODE 0 branching: aggregate inputs loaded only for qualifying rows;
+            // MODE 1 predicated aggregation: loaded for every row, x predicate;
+            // MODE 2 predicated lookups: gathers read position fk*pred (slot 0)
+            if (MODE == 0 ? ok : valid) {
+                const int64_t pm = ok ? 1 : 0;
 #pragma unroll
                 for (int g = 0; g < VD_MAX_AGGS; ++g) {
                     if (g >= NA) break;
                     int64_t pr = 1;
                     if (a.a_kind[g] != VD_AGG_COUNT) {
+                        bool e = false;
                         for (int f = 0; f < a.a_nf[g]; ++f) {
                             int64_t x = 0;
-                            if (a.a_col[g][f] >= 0) x = gf_fetch(a, w, a.a_col[g][f]).i;
+                            if (a.a_col[g][f] >= 0) {
+                                Val v = gf_fetch(a, w, a.a_col[g][f], MODE == 2 && !ok);
+                                e |= v.eps;
+                                x = v.i;
+                            }
                             pr *= a.a_a[g][f] + a.a_b[g][f] * x;
                         }
+                        if (e) pr = 0;  // an epsilon input is skipped by the fold (A5)
                     }
-                    racc[g] += pr;
+                    racc[g] += (MODE == 0) ? pr : pr * pm;
                 }
-                racc[VD_MAX_AGGS] += 1;
+                racc[VD_MAX_AGGS] += pm;
             }
             return;
         }
@@ -1225,11 +1240,17 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
             for (int g = 0; g < NA; ++g) {
                 int64_t pr = 1;
                 if (a.a_kind[g] != VD_AGG_COUNT) {
+                    bool e = false;
                     for (int f = 0; f < a.a_nf[g]; ++f) {
                         int64_t x = 0;
-                        if (a.a_col[g][f] >= 0) x = gf_fetch(a, w, a.a_col[g][f]).i;
+                        if (a.a_col[g][f] >= 0) {
+                            Val v = gf_fetch(a, w, a.a_col[g][f]);
+                            e |= v.eps;
+                            x = v.i;
+                        }
                         pr *= a.a_a[g][f] + a.a_b[g][f] * x;
                     }
+                    if (e) pr = 0;  // an epsilon input is skipped by the fold (A5)
                 }
                 sv[g] = pr;
             }
@@ -1498,6 +1519,180 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
             t += get_i128(x);
         }
         put_i128(&out[k], t);
+    }
+}
+
+// ============================================================================
+// Star-join scalar fragment (Q19 shape, C5): lineitem x part through a dense
+// FK, a disjunction of conjunctions whose terms fall into fixed slots --
+//   base  : two u8 set-membership slots (l_shipmode IN, l_shipinstruct IN),
+//           one i64 range slot (l_quantity)
+//   dim   : two u8 set-membership slots (p_brand, p_container), one i32
+//           range slot (p_size), gathered through the FK
+// -- and SUM(X * (a + b*Y)) + COUNT over two i64 base columns.  Only the
+// filter columns stream through the TMA ring (fk, range column, two u8
+// columns: 14 B/row); the union of every conjunction's base slots is tested
+// first, the part row is gathered only for the survivors (late
+// materialisation), and X / Y are loaded late (branching).
+// ============================================================================
+constexpr int ST_TILE = 4096;
+constexpr int ST_MAXCONJ = VD_MAX_CONJ;
+
+struct StarArgs {
+    const int32_t* fk;
+    const int64_t* rq;        // i64 range column (base)
+    const uint8_t* u1;        // u8 columns (base)
+    const uint8_t* u2;
+    const int64_t* x;         // aggregate columns (late loads)
+    const int64_t* y;
+    const uint8_t* d1;        // u8 columns (dimension, gathered)
+    const uint8_t* d2;
+    const int32_t* dr;        // i32 range column (dimension, gathered)
+    int64_t dim_len, bias;
+    int32_t nconj;
+    // lut[k][code]: bit c set <=> code passes conjunction c's terms on u8 slot k
+    // (k = 0,1 base, 2,3 dimension); an epsilon code passes only a slot the
+    // conjunction does not constrain (reading A9)
+    uint8_t lut[4][256];
+    int64_t rq_lo[ST_MAXCONJ], rq_hi[ST_MAXCONJ];
+    int32_t dr_lo[ST_MAXCONJ], dr_hi[ST_MAXCONJ];
+    int64_t a, b;
+    int32_t nstages;
+    int64_t n;
+    int32_t sum_slot, cnt_slot, naggs;
+};
+
+template <bool NARROW>
+__global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_star(const __grid_constant__ StarArgs a, int64_t ntiles,
+                                                              Slot16* __restrict__ parts,
+                                                              unsigned int* __restrict__ done,
+                                                              Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    constexpr int SB = ST_TILE * (4 + 8 + 1 + 1);
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * SB);
+    uint64_t* empty = full + a.nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < a.nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], FKG_CW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    __shared__ uint32_t s_lut[4][64];  // the four LUTs, byte-addressed
+    for (int i = threadIdx.x; i < 256; i += blockDim.x)
+        s_lut[i >> 6][i & 63] = reinterpret_cast<const uint32_t*>(&a.lut[0][0])[i];
+    __syncthreads();
+    const uint8_t* L = reinterpret_cast<const uint8_t*>(&s_lut[0][0]);
+    int64_t sum = 0, cnt = 0;
+    auto row = [&](int64_t r, int32_t fk, int64_t rq, uint32_t u1, uint32_t u2) {
+        uint32_t m = L[u1] & L[256 + u2];
+        if (!m) return;  // most rows stop here: two shared-memory byte lookups
+#pragma unroll
+        for (int c = 0; c < ST_MAXCONJ; ++c)
+            if (!(rq >= a.rq_lo[c] && rq <= a.rq_hi[c])) m &= ~(1u << c);
+        if (!m) return;
+        const int64_t p = (int64_t)fk - a.bias;
+        // late gather of the dimension row (only for base-qualified rows); a
+        // position outside the dimension gathers epsilon (reading A9)
+        uint32_t d1 = 0xFF, d2 = 0xFF;
+        int32_t dr = INT32_MIN;
+        if (fk != INT32_MIN && p >= 0 && p < a.dim_len) {
+            d1 = __ldg(a.d1 + p);
+            d2 = __ldg(a.d2 + p);
+            dr = __ldg(a.dr + p);
+        }
+        m &= L[512 + d1] & L[768 + d2];
+#pragma unroll
+        for (int c = 0; c < ST_MAXCONJ; ++c)
+            if (!(dr >= a.dr_lo[c] && dr <= a.dr_hi[c])) m &= ~(1u << c);
+        if (!m) return;
+        const int64_t x = __ldg(a.x + r), y = __ldg(a.y + r);  // late loads
+        cnt += 1;
+        if (x == INT64_MIN || y == INT64_MIN) return;  // epsilon factor: contributes nothing
+        if (NARROW) sum += (int64_t)(int32_t)x * (int64_t)(int32_t)((uint32_t)a.a + (uint32_t)a.b * (uint32_t)y);
+        else sum += x * (a.a + a.b * y);
+    };
+    if (warp == FKG_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % a.nstages);
+                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * SB;
+                const int64_t r0 = tile * ST_TILE;
+                mbar_expect_tx(&full[s], SB);
+                tma_load_1d(st, a.fk + r0, ST_TILE * 4, &full[s], pol);
+                tma_load_1d(st + ST_TILE * 4, a.rq + r0, ST_TILE * 8, &full[s], pol);
+                tma_load_1d(st + ST_TILE * 12, a.u1 + r0, ST_TILE, &full[s], pol);
+                tma_load_1d(st + ST_TILE * 13, a.u2 + r0, ST_TILE, &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % a.nstages);
+            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            const uint8_t* st = smem + (size_t)s * SB;
+            constexpr int RPT = ST_TILE / FKG_NT;
+            int32_t f[RPT];
+            int64_t q[RPT];
+            uint32_t m1[RPT], m2[RPT];
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) {
+                const int r = threadIdx.x + k * FKG_NT;
+                f[k] = reinterpret_cast<const int32_t*>(st)[r];
+                q[k] = reinterpret_cast<const int64_t*>(st + ST_TILE * 4)[r];
+                m1[k] = st[ST_TILE * 12 + r];
+                m2[k] = st[ST_TILE * 13 + r];
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) row(tile * ST_TILE + threadIdx.x + k * FKG_NT, f[k], q[k], m1[k], m2[k]);
+        }
+        if (blockIdx.x == 0)
+            for (int64_t r = ntiles * ST_TILE + threadIdx.x; r < a.n; r += FKG_NT) row(r, a.fk[r], a.rq[r], a.u1[r], a.u2[r]);
+    }
+    // warp (int64 proven) -> CTA (int128) -> grid
+    __shared__ i128 s_w[FKG_THREADS / 32][2];
+    const int64_t ws_ = warp_sum_i64(sum), wc = warp_sum_i64(cnt);
+    if (lane == 0) { s_w[warp][0] = ws_; s_w[warp][1] = wc; }
+    __syncthreads();
+    if (threadIdx.x < 2) {
+        i128 t = 0;
+        for (int w = 0; w < FKG_THREADS / 32; ++w) t += s_w[w][threadIdx.x];
+        put_i128(&parts[(size_t)blockIdx.x * 2 + threadIdx.x], t);
+    }
+    __shared__ bool s_last;
+    __shared__ Slot16 s_raw2[2];
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < 2) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
+            t += get_i128(x);
+        }
+        put_i128(&s_raw2[threadIdx.x], t);
+    }
+    __syncthreads();
+    if (threadIdx.x <= a.naggs) {
+        const int src = (threadIdx.x == a.naggs || threadIdx.x == a.cnt_slot) ? 1 : 0;
+        out[threadIdx.x] = s_raw2[src];
     }
 }
 
@@ -2194,6 +2389,163 @@ static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols,
     return VD_OK;
 }
 
+// ---- star-join (Q19 shape) matching -------------------------------------------------
+static vd_status try_star(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                          void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    const char* var = getenv("VD_STAR_VARIANT");
+    if (var && strcmp(var, "off") == 0) return VD_OK;
+    if (p->nkeyparts != 0 || p->ngroups != 1 || p->pred.nconj < 1 || p->pred.nconj > ST_MAXCONJ) return VD_OK;
+    if (p->ngathers < 1 || p->ngathers > 3) return VD_OK;
+    const int fkcol = p->gathers[0].fk_col;
+    for (int g = 0; g < p->ngathers; ++g)
+        if (p->gathers[g].fk_col != fkcol || p->gathers[g].bias != p->gathers[0].bias) return VD_OK;
+    if (cols[fkcol].dtype != VD_I32) return VD_OK;
+    int64_t dim_len = dims[p->gathers[0].dim_col].len;
+    for (int g = 0; g < p->ngathers; ++g)
+        if (dims[p->gathers[g].dim_col].len != dim_len) return VD_OK;
+    // slot assignment by column: base u8 sets (2), base i64 range (1), dim u8 sets (2), dim i32 range (1)
+    int bu[2] = {-1, -1}, br = -1, du[2] = {-1, -1}, dr = -1;
+    auto dt_of = [&](int c) { return c < ncols ? cols[c].dtype : dims[p->gathers[c - ncols].dim_col].dtype; };
+    auto take = [](int* slot, int nslot, int c) {
+        for (int k = 0; k < nslot; ++k) { if (slot[k] == c) return true; if (slot[k] < 0) { slot[k] = c; return true; } }
+        return false;
+    };
+    for (int c = 0; c < p->pred.nconj; ++c)
+        for (int t = 0; t < p->pred.conj[c].nterms; ++t) {
+            const vd_term& tm = p->pred.conj[c].terms[t];
+            const int dt = dt_of(tm.col);
+            const bool base = tm.col < ncols;
+            bool ok;
+            if (dt == VD_U8) ok = base ? take(bu, 2, tm.col) : take(du, 2, tm.col);
+            else if (base && dt == VD_I64) ok = take(&br, 1, tm.col);
+            else if (!base && dt == VD_I32) ok = take(&dr, 1, tm.col);
+            else ok = false;
+            if (!ok) return VD_OK;
+        }
+    StarArgs A;
+    std::memset(&A, 0, sizeof(A));
+    A.nconj = p->pred.nconj;
+    const int uslot[4] = {bu[0], bu[1], du[0], du[1]};
+    for (int c = 0; c < ST_MAXCONJ; ++c) {
+        int64_t rlo = INT64_MIN, rhi = INT64_MAX, dlo = INT32_MIN, dhi = INT32_MAX;
+        if (c >= A.nconj) {  // unused conjunction: never passes
+            A.rq_lo[c] = 1; A.rq_hi[c] = 0; A.dr_lo[c] = 1; A.dr_hi[c] = 0;
+            continue;
+        }
+        bool ucon[4] = {false, false, false, false};
+        bool pass[4][256];
+        for (int k = 0; k < 4; ++k) std::fill(pass[k], pass[k] + 256, true);
+        for (int t = 0; t < p->pred.conj[c].nterms; ++t) {
+            const vd_term& tm = p->pred.conj[c].terms[t];
+            bool ok = true;
+            int k = -1;
+            for (int q = 0; q < 4; ++q) if (uslot[q] == tm.col) k = q;
+            if (k >= 0) {
+                ucon[k] = true;
+                for (int x = 0; x < 256; ++x) {
+                    bool r;
+                    switch (tm.cmp) {
+                    case VD_CMP_GT: r = x > tm.ival; break;
+                    case VD_CMP_LT: r = x < tm.ival; break;
+                    case VD_CMP_EQ: r = x == tm.ival; break;
+                    case VD_CMP_GE: r = x >= tm.ival; break;
+                    case VD_CMP_LE: r = x <= tm.ival; break;
+                    case VD_CMP_NE: r = x != tm.ival; break;
+                    case VD_CMP_IN: r = x < 64 && (((uint64_t)tm.ival >> x) & 1ull); break;
+                    default: return VD_OK;
+                    }
+                    pass[k][x] = pass[k][x] && r;
+                }
+            } else if (tm.col == br) {
+                ok = term_interval(tm, &rlo, &rhi);
+                rlo = std::max<int64_t>(rlo, INT64_MIN + 1);  // epsilon never passes a term
+            } else if (tm.col == dr) {
+                ok = term_interval(tm, &dlo, &dhi);
+                dlo = std::max<int64_t>(dlo, INT32_MIN + 1);
+            } else {
+                ok = false;
+            }
+            if (!ok) return VD_OK;
+        }
+        for (int k = 0; k < 4; ++k) {
+            if (ucon[k]) pass[k][255] = false;
+            for (int x = 0; x < 256; ++x)
+                if (pass[k][x]) A.lut[k][x] |= (uint8_t)(1u << c);
+        }
+        A.rq_lo[c] = rlo; A.rq_hi[c] = rhi;
+        A.dr_lo[c] = (int32_t)std::max<int64_t>(dlo, INT32_MIN);
+        A.dr_hi[c] = (int32_t)std::min<int64_t>(dhi, INT32_MAX);
+        if (dlo > INT32_MAX || dhi < INT32_MIN) { A.dr_lo[c] = 1; A.dr_hi[c] = 0; }
+    }
+    // aggregates
+    A.sum_slot = A.cnt_slot = -1;
+    A.naggs = p->naggs;
+    int X = -1, Y = -1;
+    for (int g = 0; g < p->naggs; ++g) {
+        const vd_agg& ag = p->aggs[g];
+        if (ag.kind == VD_AGG_COUNT) { if (A.cnt_slot >= 0) return VD_OK; A.cnt_slot = g; continue; }
+        if (ag.kind != VD_AGG_SUM || A.sum_slot >= 0 || ag.nfactors != 2 || !plain_col(ag.f[0])) return VD_OK;
+        X = ag.f[0].col;
+        Y = ag.f[1].col;
+        if (X >= ncols || Y < 0 || Y >= ncols || cols[X].dtype != VD_I64 || cols[Y].dtype != VD_I64) return VD_OK;
+        A.a = ag.f[1].a;
+        A.b = ag.f[1].b;
+        A.sum_slot = g;
+    }
+    if (A.sum_slot < 0) return VD_OK;
+    // slots the predicate does not use read a claimed column through an all-pass LUT
+    const int cu1 = bu[0], cu2 = bu[1] >= 0 ? bu[1] : bu[0];
+    if (cu1 < 0 || br < 0) return VD_OK;  // the base prefilter needs a u8 and the i64 column
+    for (int c : {fkcol, br, cu1, cu2})
+        if (((uintptr_t)cols[c].data % 16) != 0) return VD_OK;
+    Bound bx = col_bound(p, cols, ncols, dims, X), by = col_bound(p, cols, ncols, dims, Y);
+    if (!bx.known || !by.known) return VD_OK;
+    vd_factor fy;
+    fy.col = Y; fy.a = A.a; fy.b = A.b;
+    const double fmx = factor_absmax(fy, by), xmx = std::max(std::fabs(bx.lo), std::fabs(bx.hi));
+    const int grid = num_sms();
+    const double rows_per_thread = std::ceil((double)n / ((double)grid * FKG_NT)) + ST_TILE;
+    if (xmx * fmx * rows_per_thread >= 9.0e18) return VD_OK;
+    const bool narrow = xmx < 2147483647.0 && fmx < 2147483647.0 && std::fabs((double)A.a) < 2.0e9 &&
+                        std::fabs((double)A.b) < 2.0e9 && std::max(std::fabs(by.lo), std::fabs(by.hi)) < 2147483647.0;
+    A.fk = (const int32_t*)cols[fkcol].data;
+    A.rq = (const int64_t*)cols[br].data;
+    A.u1 = (const uint8_t*)cols[cu1].data;
+    A.u2 = (const uint8_t*)cols[cu2].data;
+    A.x = (const int64_t*)cols[X].data;
+    A.y = (const int64_t*)cols[Y].data;
+    auto dimptr = [&](int c) { return dims[p->gathers[c - ncols].dim_col].data; };
+    const int cd1 = du[0], cd2 = du[1] >= 0 ? du[1] : du[0];
+    if (cd1 < 0 || dr < 0) return VD_OK;
+    A.d1 = (const uint8_t*)dimptr(cd1);
+    A.d2 = (const uint8_t*)dimptr(cd2);
+    A.dr = (const int32_t*)dimptr(dr);
+    A.dim_len = dim_len;
+    A.bias = p->gathers[0].bias;
+    A.n = n;
+    constexpr size_t SB = ST_TILE * 14;
+    A.nstages = (int)std::min<size_t>(GF_MAXSTAGES, (200 * 1024) / SB);
+    const size_t smem = (size_t)A.nstages * SB + 2 * A.nstages * 8;
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    if (narrow) {
+        cudaFuncSetAttribute(k_pipe_star<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_star<true><<<grid, FKG_THREADS, smem, s>>>(A, n / ST_TILE, parts, dn, (Slot16*)out);
+    } else {
+        cudaFuncSetAttribute(k_pipe_star<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_star<false><<<grid, FKG_THREADS, smem, s>>>(A, n / ST_TILE, parts, dn, (Slot16*)out);
+    }
+    ++*nl;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    set_fragment("star_join");
+    *done = true;
+    return VD_OK;
+}
+
 // ---- gather-fold matching -------------------------------------------------------
 static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
                         void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
@@ -2346,12 +2698,14 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
     Slot16* rawp = (Slot16*)out;
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-    const int mode = p->sel_mode == VD_SEL_PREDICATED ? 1 : 0;
+    const int mode = p->sel_mode == VD_SEL_PREDICATED ? 1 : (p->sel_mode == VD_SEL_PREDICATED_LOOKUP ? 2 : 0);
 #define GF_LAUNCH(M, SC)                                                                              \
     cudaFuncSetAttribute(k_pipe_gf<M, SC>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);    \
     k_pipe_gf<M, SC><<<grid, GF_THREADS, smem, s>>>(A, n / GF_TILE, parts, dn, rawp);
     const bool scalar = p->ngroups == 1;
-    if (mode) {
+    if (mode == 2) {
+        if (scalar) { GF_LAUNCH(2, true) } else { GF_LAUNCH(0, false) }  // grouped: lookups are per qualifying row
+    } else if (mode == 1) {
         if (scalar) { GF_LAUNCH(1, true) } else { GF_LAUNCH(1, false) }
     } else {
         if (scalar) { GF_LAUNCH(0, true) } else { GF_LAUNCH(0, false) }
@@ -2476,6 +2830,8 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_fkg(p, cols, ncols, n, dims, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+        st = try_star(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;

@@ -508,6 +508,7 @@ vd_status vd_run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_
     if (plan->ngathers < 0 || plan->ngathers > VD_MAX_GATHERS) { set_error("pipeline: ngathers in [0, 4]"); return VD_E_ARG; }
     if (plan->nkeyparts < 0 || plan->nkeyparts > VD_MAX_KEYPARTS) { set_error("pipeline: nkeyparts in [0, 3]"); return VD_E_ARG; }
     if (plan->nkeyparts == 0 && plan->ngroups != 1) { set_error("pipeline: scalar plans have ngroups = 1"); return VD_E_ARG; }
+    if (plan->sel_mode < VD_SEL_BRANCH || plan->sel_mode > VD_SEL_PREDICATED_LOOKUP) { set_error("pipeline: sel_mode"); return VD_E_ARG; }
     if (plan->ngathers > 0 && (!dims || ndims < 1)) { set_error("pipeline: gathers need dims"); return VD_E_NULL; }
     vd_status st;
     for (int c = 0; c < ncols; ++c)

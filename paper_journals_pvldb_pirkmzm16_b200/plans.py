@@ -75,3 +75,18 @@ def q9(sel_mode=VD_SEL_BRANCH, force_generic=False):
     nation*7 + (year(l_shipdate) - 1992) (175 groups), sum(ext*(100-disc)), count."""
     return pipeline(sel_mode=sel_mode, gathers=[(0, 0, 1)], key=[(4, 0, 0, 7), (1, 1, 1992, 1)], ngroups=175,
                     aggs=[("sum", [2, (3, 100, -1)]), ("count",)], force_generic=force_generic)
+
+
+# Fig 16 selective FK join: a 128 MB target (16 M int64 rows), larger than the 126 MB L2
+FKJSEL_TARGET_ROWS = 16 * 1024 * 1024
+FKJSEL_VMAX = 1_000_000
+
+
+def fkjsel(threshold: int, sel_mode=VD_SEL_BRANCH, force_generic=False):
+    """Selective FK join (Fig 16): SELECT sum(target.v) FROM
+    fact, target WHERE fact.fk = target.pk AND fact.v < threshold.  Columns:
+    fact [fk (int32, 1-based), v (int32)], dims [target.v (int64)].  The
+    three strategies of Fig 16 are sel_mode BRANCH / PREDICATED (predicated
+    aggregation) / PREDICATED_LOOKUP (position x predicate)."""
+    return pipeline(pred_=pred([[(1, "<", int(threshold))]]), sel_mode=sel_mode, gathers=[(0, 0, 1)],
+                    aggs=[("sum", [2]), ("count",)], force_generic=force_generic)

@@ -30,7 +30,7 @@ VD_OK, VD_E_NULL, VD_E_DTYPE, VD_E_SHAPE, VD_E_CTRL, VD_E_DOMAIN, VD_E_OVERFLOW,
     VD_E_UNSUPPORTED, VD_E_ARG = range(11)
 VD_U8, VD_I32, VD_I64, VD_F32, VD_F64 = range(5)
 VD_CMP_GT, VD_CMP_LT, VD_CMP_EQ, VD_CMP_GE, VD_CMP_LE, VD_CMP_NE, VD_CMP_IN = range(7)
-VD_SEL_BRANCH, VD_SEL_PREDICATED = 0, 1
+VD_SEL_BRANCH, VD_SEL_PREDICATED, VD_SEL_PREDICATED_LOOKUP = 0, 1, 2
 VD_OP_SELECT, VD_OP_FOLD, VD_OP_SCATTER, VD_OP_PIPELINE, VD_OP_FOLD_SELECT, VD_OP_PARTITION = range(6)
 VD_AGG_SUM, VD_AGG_COUNT, VD_AGG_MIN, VD_AGG_MAX = range(4)
 VD_SCATTER_UNIQUE = 1

@@ -3,6 +3,7 @@
 
   python scripts/sweep.py fig1  > gpurun_out/sweep_fig1.jsonl   # C2: 1e9 f32 -> positions
   python scripts/sweep.py fig15 > gpurun_out/sweep_fig15.jsonl  # selective aggregation (select + FoldSum)
+  python scripts/sweep.py fig16 > gpurun_out/sweep_fig16.jsonl  # selective FK join: branch / predicated / lookup
 
 Fig 1 and Fig 15: branching vs
 predicated (cursor arithmetic) over selectivities 1..100 % (plus the Fig 15
@@ -48,9 +49,10 @@ def main():
     what = sys.argv[1]
     if what == "table":
         return table(sys.argv[2:])
-    workload = {"fig1": "selpos", "fig15": "select"}[what]
+    workload = {"fig1": "selpos", "fig15": "select", "fig16": "fkjsel"}[what]
+    modes = ["branch", "predicated", "lookup"] if what == "fig16" else ["branch", "predicated"]
     for s in SEL:
-        for mode in ["branch", "predicated"]:
+        for mode in modes:
             print(json.dumps(run(workload, s, mode, 30 if workload == "selpos" else 100)), flush=True)
 
 

@@ -151,8 +151,146 @@ def test_fkj_q19_vs_oracle(sel_mode, generic, n):
     dkeep, dviews = load([part[c] for c in plans.Q19_DIMS])
     plan = plans.q19(codes(), sel_mode, force_generic=generic)
     got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews,
-                                 want=("generic",) if generic else ("gather_fold",))[0], plan)
+                                 want=("generic",) if generic else ("star_join",))[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
+def test_fkj_q19_gather_fold_fragment():
+    """The Q19 plan through the general gather-fold fragment (star-join off)."""
+    import os
+    sf = 0.05
+    li = lineitem(sf, 300007)
+    part, supp = _dims(sf)
+    exp = oracle.fkj(0, li, part, supp)
+    keep, views = load([li[c] for c in plans.Q19_COLS])
+    dkeep, dviews = load([part[c] for c in plans.Q19_DIMS])
+    os.environ["VD_STAR_VARIANT"] = "off"
+    try:
+        got = vd.decode_partials(run(plans.q19(codes()), views, len(li["l_partkey"]), dviews,
+                                     want=("gather_fold",))[0], plans.q19(codes()))
+    finally:
+        del os.environ["VD_STAR_VARIANT"]
+    assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
+def _term_expr(name, col, cmp, c, out):
+    """A predicate term as the oracle's Greater/Equals/LogicalOr (reading A8)."""
+    if cmp == ">":
+        out.append(f"{name} := Greater({col}, {c})")
+    elif cmp == "<":
+        out.append(f"{name} := Greater({c}, {col})")
+    elif cmp == "==":
+        out.append(f"{name} := Equals({col}, {c})")
+    elif cmp == ">=":
+        out.append(f"{name} := Greater({col}, {c - 1})")
+    elif cmp == "<=":
+        out.append(f"{name} := Greater({c + 1}, {col})")
+    elif cmp == "!=":
+        out += [f"{name}_a := Greater({col}, {c})", f"{name}_b := Greater({c}, {col})",
+                f"{name} := LogicalOr({name}_a, {name}_b)"]
+    else:  # in: c is a list of codes
+        codes = c or [1000]  # the empty set: never equal
+        out.append(f"{name} := Equals({col}, {codes[0]})")
+        for k, v in enumerate(codes[1:]):
+            out += [f"{name}_{k} := Equals({col}, {v})", f"{name} := LogicalOr({name}, {name}_{k})"]
+
+
+@pytest.mark.parametrize("seed", range(12))
+def test_star_join_random_predicates_vs_oracle(seed):
+    """Star-join fragment on random disjunctive predicates over its slot
+    columns (every comparison kind, dictionary codes >= 64, epsilon in every
+    column, FKs outside the dimension, conjunctions without dimension terms)
+    against the oracle: each conjunction's FoldSelect positions from an oracle
+    program (a term over epsilon is false, A9), their union, then the oracle's
+    Gather -> Multiply -> FoldSum / FoldCount over it."""
+    rng = np.random.default_rng(100 + seed)
+    n, m = 70001 + seed * 997, 3001
+    fk = rng.integers(-3, m + 5, n).astype(np.int32)
+    rq = rng.integers(0, 6000, n).astype(np.int64)
+    u1 = rng.integers(0, 90, n).astype(np.uint8)
+    u2 = rng.integers(0, 8, n).astype(np.uint8)
+    x = rng.integers(0, 10**7, n).astype(np.int64)
+    y = rng.integers(0, 11, n).astype(np.int64)
+    d1 = rng.integers(0, 80, m).astype(np.uint8)
+    d2 = rng.integers(0, 40, m).astype(np.uint8)
+    dr = rng.integers(1, 51, m).astype(np.int32)
+    eps = {}
+    for nm, arr, e in [("fk", fk, -2**31), ("rq", rq, -2**63), ("u1", u1, 255), ("u2", u2, 255), ("x", x, -2**63),
+                       ("y", y, -2**63), ("d1", d1, 255), ("d2", d2, 255), ("dr", dr, -2**31)]:
+        msk = rng.random(arr.size) < 0.01
+        arr[msk] = e
+        eps[nm] = msk
+    base = {"fk": fk, "rq": rq, "x": x, "y": y, "u1": u1, "u2": u2}  # plan column order
+    cols = list(base)
+    slot_ref = {"rq": 1, "u1": 4, "u2": 5, "d1": 6, "d2": 7, "dr": 8}
+
+    def rand_term(colname):
+        if colname in ("u1", "u2", "d1", "d2"):
+            cmp = str(rng.choice([">", "<", "==", ">=", "<=", "!=", "in"], p=[.17, .17, .04, .17, .17, .14, .14]))
+            if cmp == "in":
+                return cmp, sorted(set(int(v) for v in rng.integers(0, 64, rng.integers(0, 60))))
+            return cmp, int(rng.integers(0, 90))
+        hi = 6000 if colname == "rq" else 50
+        return str(rng.choice([">", "<", "==", ">=", "<="], p=[.3, .3, .05, .175, .175])), int(rng.integers(0, hi))
+
+    nconj = int(rng.integers(1, 5))
+    conjs = []
+    for c in range(nconj):
+        names = [k for k in slot_ref if rng.random() < 0.4] or ["u2"]
+        if c == 0:
+            names = sorted(set(names) | {"u1", "rq", "d1", "dr"})
+        conjs.append([(k, *rand_term(k)) for k in names for _ in range(1 + int(rng.random() < 0.2))][:8])
+    # the oracle: one program per conjunction, union of the selected positions
+    sel = np.zeros(n, dtype=bool)
+    inputs = {f"fact__{k}": (v, eps[k]) for k, v in base.items()}
+    inputs.update({f"dim__{k}": (v, eps[k]) for k, v in (("d1", d1), ("d2", d2), ("dr", dr))})
+    for c, terms in enumerate(conjs):
+        lines = ["p := Subtract(fact.fk, 1)", "gd1 := Gather(dim.d1, p)", "gd2 := Gather(dim.d2, p)",
+                 "gdr := Gather(dim.dr, p)"]
+        ref = {"rq": "fact.rq", "u1": "fact.u1", "u2": "fact.u2", "d1": "gd1", "d2": "gd2", "dr": "gdr"}
+        names = []
+        for k, (colname, cmp, val) in enumerate(terms):
+            _term_expr(f"t{k}", ref[colname], cmp, val, lines)
+            names.append(f"t{k}")
+        lines.append(f"a := LogicalAnd({names[0]}, {names[0]})")
+        for nm in names[1:]:
+            lines.append(f"a := LogicalAnd(a, {nm})")
+        lines.append("pos := FoldSelect(a)")
+        pos, pe = oracle.run("\n".join(lines), **inputs).get_arrays("pos")
+        sel[pos[~pe]] = True
+    upos = np.nonzero(sel)[0].astype(np.int64)
+    agg = oracle.run("""
+    gx := Gather(fact.x, pos)
+    gy := Gather(fact.y, pos)
+    f := Multiply(gy, -1)
+    t := Add(f, 100)
+    pr := Multiply(gx, t)
+    s := FoldSum(pr)
+    c := FoldCount(pos)
+    """, fact__x=(x, eps["x"]), fact__y=(y, eps["y"]), pos=upos)
+    exp_s, exp_c = (agg.get("s")[0], agg.get("c")[0]) if upos.size else (0, 0)
+    # the GPU plan
+    vconj = []
+    for terms in conjs:
+        ts = []
+        for colname, cmp, val in terms:
+            if cmp == "in":
+                ts.append((slot_ref[colname], "in", val))
+            else:
+                ts.append((slot_ref[colname], str(cmp), val))
+        vconj.append(ts)
+    keep, views = load([base[k] for k in cols])
+    dkeep, dviews = load([d1, d2, dr])
+    plan = vd.pipeline(pred_=vd.pred(vconj), gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)],
+                       aggs=[("sum", [2, (3, 100, -1)]), ("count",)])
+    got = vd.decode_partials(run(plan, views, n, dviews, want=("star_join",))[0], plan)
+    if exp_c == 0:
+        assert got == {}
+    else:
+        assert got == {0: [int(exp_s), int(exp_c), int(exp_c)]}
+    gen_plan = vd.pipeline(pred_=vd.pred(vconj), gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)],
+                           aggs=[("sum", [2, (3, 100, -1)]), ("count",)], force_generic=True)
+    assert vd.decode_partials(run(gen_plan, views, n, dviews, want=("generic",))[0], gen_plan) == got
 
 
 @pytest.mark.parametrize("sel_mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED])
@@ -262,3 +400,36 @@ def test_fkj_q9_gather_fold_fragment(variant):
     finally:
         del os.environ["VD_FKG_VARIANT"]
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
+@pytest.mark.parametrize("mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED, vd.VD_SEL_PREDICATED_LOOKUP])
+@pytest.mark.parametrize("sel", [0.0, 0.013, 0.5, 1.0])
+def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel):
+    """Fig 16: branching, predicated aggregation and predicated
+    lookups give the same SUM(target.v) and count as the oracle's program
+    Gather(target.v, fk - 1) -> FoldSelect(v < t) -> FoldSum."""
+    n, m = 100003, 5000
+    rng = np.random.default_rng(7)
+    fk = rng.integers(1, m + 1, n).astype(np.int32)
+    v = rng.integers(0, plans.FKJSEL_VMAX, n).astype(np.int32)
+    tv = rng.integers(-10**6, 10**6, m).astype(np.int64)
+    thr = int(round(sel * plans.FKJSEL_VMAX))
+    prog = f"""
+    p := Subtract(fact.fk, 1)
+    g := Gather(target.v, p)
+    q := Greater({thr}, fact.v)
+    pos := FoldSelect(q)
+    sel := Gather(g, pos)
+    s := FoldSum(sel)
+    c := FoldCount(sel)
+    """
+    po = oracle.run(prog, fact__fk=fk, fact__v=v, target__v=tv)
+    exp_s, exp_c = po.get("s")[0], po.get("c")[0]
+    keep, views = load([fk, v])
+    dkeep, dviews = load([tv])
+    plan = plans.fkjsel(thr, mode)
+    got = vd.decode_partials(run(plan, views, n, dviews, want=("gather_fold",))[0], plan)
+    if exp_c == 0:
+        assert got == {}
+    else:
+        assert got == {0: [exp_s, exp_c, exp_c]}
