@@ -63,7 +63,8 @@ def parse():
 
 
 def default_sf(w):
-    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0}[w]
+    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0,
+            "select_unfused": 0.0}[w]
 
 
 # ---------------------------------------------------------------------------

@@ -1382,14 +1382,18 @@ struct FkgArgs {
     int32_t naggs;
 };
 
-template <bool NARROW>
+template <bool NARROW, bool ATOM, bool PIPE>
 __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_constant__ FkgArgs a, int64_t ntiles,
                                                             Slot16* __restrict__ parts, unsigned int* __restrict__ done,
                                                             Slot16* __restrict__ out) {
     extern __shared__ __align__(128) uint8_t smem[];
     constexpr int SB = FKG_TILE * (4 + 4 + 8 + 8);
-    int64_t* acc = reinterpret_cast<int64_t*>(smem + (size_t)a.nstages * SB);  // [FKG_CW][ngroups][2]
-    int64_t* sv = acc + (size_t)FKG_CW * a.ngroups * 2;                        // [FKG_CW][32]
+    // per-warp group slots as three u32 arrays (sum low word, sum high word,
+    // count) so that random keys spread over all 32 banks; + a trash slot
+    const int GS = a.ngroups + 1;
+    const int GSP = (GS + 31) & ~31;
+    uint32_t* acc = reinterpret_cast<uint32_t*>(smem + (size_t)a.nstages * SB);  // [FKG_CW][3][GSP]
+    int64_t* sv = reinterpret_cast<int64_t*>(acc + (size_t)FKG_CW * 3 * GSP);   // [FKG_CW][32]
     int16_t* ytab = reinterpret_cast<int16_t*>(sv + FKG_CW * 32);
     uint64_t* full = reinterpret_cast<uint64_t*>(ytab + ((a.ydays + 7) & ~7));
     uint64_t* empty = full + a.nstages;
@@ -1401,34 +1405,59 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
         }
         fence_mbar_init();
     }
-    for (int k = threadIdx.x; k < FKG_CW * a.ngroups * 2; k += FKG_THREADS) acc[k] = 0;
+    for (int k = threadIdx.x; k < FKG_CW * 3 * GSP; k += FKG_THREADS) acc[k] = 0;
     for (int k = threadIdx.x; k < a.ydays; k += FKG_THREADS) ytab[k] = (int16_t)year_of_day(a.ylo + k);
     __syncthreads();
-    int64_t* wacc = acc + (size_t)warp * a.ngroups * 2;
+    uint32_t* wlo = acc + (size_t)warp * 3 * GSP;
+    uint32_t* whi = wlo + GSP;
+    uint32_t* wcnt = whi + GSP;
     int64_t* wsv = sv + warp * 32;
 
-    // one 32-row step of a warp: lane's row (fk, kb, x, y), valid flag
-    auto step = [&](bool valid, int32_t fk, int32_t kb, int64_t x, int64_t y) {
+    // phase 1 of a 32-row step: the lane's key (-1: no group) and value; the
+    // dimension gather is issued here, so the RPT gathers of a tile are in
+    // flight together
+    // the dimension value of a row (0x100: no dimension row -- epsilon FK or
+    // outside the dimension, reading A9/A11); issued early, consumed late
+    auto gather = [&](bool valid, int32_t fk) -> int {
+        const int64_t p = (int64_t)fk - a.bias;
+        return (valid && fk != INT32_MIN && p >= 0 && p < a.dim_len) ? (int)__ldg(a.dim + p) : 0x100;
+    };
+    // the group key (-1: no group) and value of a row, given its dimension value
+    auto keyof = [&](int d, int32_t kb, int64_t x, int64_t y, int64_t& v) {
         int key = -1;
-        int64_t v = 0;
-        if (valid) {
-            const int64_t p = (int64_t)fk - a.bias;
-            if (p >= 0 && p < a.dim_len && fk != INT32_MIN) {
-                const int d = __ldg(a.dim + p);
-                int kbv = kb;
-                if (a.yfn) {
-                    const int dd = kb - a.ylo;  // the table covers [min, max] of kb (metadata)
-                    kbv = (dd >= 0 && dd < a.ydays) ? (int)ytab[dd] : -0x40000000;
-                }
-                key = (d - a.subA) * a.mA + (kbv - a.subB) * a.mB;
-                if (d == 0xFF || kb == INT32_MIN || key < 0 || key >= a.ngroups) key = -1;
-                if (NARROW) {
-                    const int32_t f = (int32_t)a.a + (int32_t)a.b * (int32_t)y;
-                    v = (int64_t)(int32_t)x * (int64_t)f;
-                } else {
-                    v = x * (a.a + a.b * y);
-                }
+        v = 0;
+        if (d != 0x100) {
+            int kbv = kb;
+            if (a.yfn) {
+                const int dd = kb - a.ylo;  // the table covers [min, max] of kb (metadata)
+                kbv = (dd >= 0 && dd < a.ydays) ? (int)ytab[dd] : -0x40000000;
             }
+            key = (d - a.subA) * a.mA + (kbv - a.subB) * a.mB;
+            if (d == 0xFF || kb == INT32_MIN || key < 0 || key >= a.ngroups) key = -1;
+            if (NARROW) {
+                const int32_t f = (int32_t)((uint32_t)a.a + (uint32_t)a.b * (uint32_t)y);
+                v = (int64_t)(int32_t)x * (int64_t)f;
+            } else {
+                v = x * (a.a + a.b * y);
+            }
+        }
+        return key;
+    };
+    // phase 2: fold the step into the warp's group slots -- shared-memory
+    // atomics (ATOM) or one leader lane per distinct key (__match_any_sync)
+    auto fold = [&](int key, int64_t v) {
+        if (ATOM) {
+            // native 32-bit shared atomics (a 64-bit one is a CAS loop): the
+            // low word returns the old value, the carry goes to the high word
+            // -- exact modulo 2^64.  Rows without a group update the trash slot.
+            const int g = key >= 0 ? key : a.ngroups;
+            const uint64_t uv = (uint64_t)v;
+            const uint32_t lo = (uint32_t)uv;
+            const uint32_t old = atomicAdd(&wlo[g], lo);
+            atomicAdd(&wcnt[g], 1u);  // < 2^32 rows per warp
+            const uint32_t hi = (uint32_t)(uv >> 32) + ((uint32_t)(old + lo) < old ? 1u : 0u);
+            if (hi) atomicAdd(&whi[g], hi);
+            return;
         }
         wsv[lane] = v;
         __syncwarp();
@@ -1436,10 +1465,36 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
         if (key >= 0 && (__ffs(m) - 1) == lane) {
             int64_t t = 0;
             for (unsigned mm = m; mm; mm &= mm - 1) t += wsv[__ffs(mm) - 1];
-            wacc[2 * key] += t;
-            wacc[2 * key + 1] += __popc(m);
+            const uint64_t cur = ((uint64_t)whi[key] << 32 | wlo[key]) + (uint64_t)t;
+            wlo[key] = (uint32_t)cur;
+            whi[key] = (uint32_t)(cur >> 32);
+            wcnt[key] += __popc(m);
         }
         __syncwarp();
+    };
+    // RPT rows at once: all low-word atomics are issued before any carry is
+    // needed, so their latencies overlap
+    constexpr int RPT = FKG_TILE / FKG_NT;
+    auto foldn = [&](const int* key, const int64_t* v) {
+        if (!ATOM) {
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) fold(key[k], v[k]);
+            return;
+        }
+        uint32_t old[RPT];
+        int g[RPT];
+#pragma unroll
+        for (int k = 0; k < RPT; ++k) {
+            g[k] = key[k] >= 0 ? key[k] : a.ngroups;
+            old[k] = atomicAdd(&wlo[g[k]], (uint32_t)(uint64_t)v[k]);
+            atomicAdd(&wcnt[g[k]], 1u);
+        }
+#pragma unroll
+        for (int k = 0; k < RPT; ++k) {
+            const uint32_t lo = (uint32_t)(uint64_t)v[k];
+            const uint32_t hi = (uint32_t)((uint64_t)v[k] >> 32) + ((uint32_t)(old[k] + lo) < old[k] ? 1u : 0u);
+            if (hi) atomicAdd(&whi[g[k]], hi);
+        }
     };
 
     if (warp == FKG_CW) {
@@ -1461,13 +1516,25 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
         }
         __syncwarp();
     } else {
+        // software pipeline: the gathers of tile i are issued, then tile i-1
+        // (whose gathers were issued one iteration earlier) is keyed and
+        // folded, so each L2 round trip overlaps a whole iteration
+        int pd[RPT], pkb[RPT];
+        int64_t px[RPT], py[RPT];
+        bool have = false;
+        auto drain = [&]() {
+            int key[RPT];
+            int64_t v[RPT];
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) key[k] = keyof(pd[k], pkb[k], px[k], py[k], v[k]);
+            foldn(key, v);
+        };
         for (int64_t it = 0;; ++it) {
             const int64_t tile = blockIdx.x + it * gridDim.x;
             if (tile >= ntiles) break;
             const int s = (int)(it % a.nstages);
             mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
             const uint8_t* st = smem + (size_t)s * SB;
-            constexpr int RPT = FKG_TILE / FKG_NT;
             int32_t f[RPT], kb[RPT];
             int64_t x[RPT], y[RPT];
 #pragma unroll
@@ -1480,14 +1547,24 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(&empty[s]);
+            int d[RPT];
 #pragma unroll
-            for (int k = 0; k < RPT; ++k) step(true, f[k], kb[k], x[k], y[k]);
+            for (int k = 0; k < RPT; ++k) d[k] = gather(true, f[k]);
+            if (PIPE && have) drain();
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) { pd[k] = d[k]; pkb[k] = kb[k]; px[k] = x[k]; py[k] = y[k]; }
+            have = true;
+            if (!PIPE) { drain(); have = false; }
         }
+        if (have) drain();
         if (blockIdx.x == 0) {
             for (int64_t base = ntiles * FKG_TILE + warp * 32; base < a.n; base += FKG_NT) {
                 const int64_t r = base + lane;
                 const bool ok = r < a.n;
-                step(ok, ok ? a.fk[r] : 0, ok ? a.kb[r] : 0, ok ? a.x[r] : 0, ok ? a.y[r] : 0);
+                int64_t v;
+                const int key = keyof(gather(ok, ok ? a.fk[r] : 0), ok ? a.kb[r] : 0, ok ? a.x[r] : 0,
+                                      ok ? a.y[r] : 0, v);
+                fold(key, v);
             }
         }
     }
@@ -1498,7 +1575,10 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
         const int g = k / (a.naggs + 1), ag = k % (a.naggs + 1);
         const int src = (ag == a.naggs || ag == a.cnt_slot) ? 1 : 0;
         i128 t = 0;
-        for (int w = 0; w < FKG_CW; ++w) t += (i128)acc[((size_t)w * a.ngroups + g) * 2 + src];
+        for (int w = 0; w < FKG_CW; ++w) {
+            const uint32_t* b = acc + (size_t)w * 3 * GSP;
+            t += src ? (i128)b[2 * GSP + g] : (i128)(int64_t)((uint64_t)b[GSP + g] << 32 | b[g]);
+        }
         put_i128(&parts[(size_t)blockIdx.x * NS + k], t);
     }
     __shared__ bool s_last;
@@ -1535,6 +1615,9 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
 // first, the part row is gathered only for the survivors (late
 // materialisation), and X / Y are loaded late (branching).
 // ============================================================================
+__device__ __forceinline__ void scalar2_finish(int64_t sum, int64_t cnt, Slot16* __restrict__ parts,
+                                               unsigned int* __restrict__ done, Slot16* __restrict__ out,
+                                               int naggs, int cnt_slot);
 constexpr int ST_TILE = 4096;
 constexpr int ST_MAXCONJ = VD_MAX_CONJ;
 
@@ -1659,18 +1742,49 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_star(const __grid_const
         if (blockIdx.x == 0)
             for (int64_t r = ntiles * ST_TILE + threadIdx.x; r < a.n; r += FKG_NT) row(r, a.fk[r], a.rq[r], a.u1[r], a.u2[r]);
     }
-    // warp (int64 proven) -> CTA (int128) -> grid
-    __shared__ i128 s_w[FKG_THREADS / 32][2];
+    scalar2_finish(sum, cnt, parts, done, out, a.naggs, a.cnt_slot);
+}
+
+// ============================================================================
+// Selective FK join fragment (Fig 16; NEXT-1):
+//   SUM(dim.v[fk - bias]) , COUNT(*)  WHERE lo <= fact.v <= hi
+// in the three strategies of Fig 16: MODE 0 branching (gather only for
+// qualifying rows), MODE 1 predicated aggregation (gather every row, x pred),
+// MODE 2 predicated lookups (gather position (fk - bias) x pred: the
+// non-qualifying rows all hit slot 0).  Each thread keeps FJ_R independent
+// gathers in flight (memory-level parallelism for the random accesses); the
+// sequential columns are read with streaming loads, coalesced per k.
+// ============================================================================
+constexpr int FJ_THREADS = 256;
+constexpr int FJ_R = 8;
+
+struct FkjsArgs {
+    const int32_t* fk;
+    const void* pv;   // predicate column (i32 / i64)
+    const void* dim;  // gathered column (i32 / i64)
+    int64_t n, dim_len, bias;
+    int64_t lo, hi;   // inclusive predicate interval (lo > epsilon)
+    int32_t naggs, sum_slot, cnt_slot;
+};
+
+// warp (int64, proven by the planner) -> CTA (int128) -> per-CTA partials ->
+// the last CTA sums them in block order and writes the plan's slot layout
+// (sum slot, count slot(s)); Fragment 2 of Fig 8 fused into the last CTA.
+__device__ __forceinline__ void scalar2_finish(int64_t sum, int64_t cnt, Slot16* __restrict__ parts,
+                                               unsigned int* __restrict__ done, Slot16* __restrict__ out,
+                                               int naggs, int cnt_slot) {
+    __shared__ i128 s_w[32][2];
+    __shared__ bool s_last;
+    __shared__ Slot16 s_raw2[2];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, nw = blockDim.x >> 5;
     const int64_t ws_ = warp_sum_i64(sum), wc = warp_sum_i64(cnt);
     if (lane == 0) { s_w[warp][0] = ws_; s_w[warp][1] = wc; }
     __syncthreads();
     if (threadIdx.x < 2) {
         i128 t = 0;
-        for (int w = 0; w < FKG_THREADS / 32; ++w) t += s_w[w][threadIdx.x];
+        for (int w = 0; w < nw; ++w) t += s_w[w][threadIdx.x];
         put_i128(&parts[(size_t)blockIdx.x * 2 + threadIdx.x], t);
     }
-    __shared__ bool s_last;
-    __shared__ Slot16 s_raw2[2];
     __syncthreads();
     if (threadIdx.x == 0) {
         __threadfence();
@@ -1690,10 +1804,195 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_star(const __grid_const
         put_i128(&s_raw2[threadIdx.x], t);
     }
     __syncthreads();
-    if (threadIdx.x <= a.naggs) {
-        const int src = (threadIdx.x == a.naggs || threadIdx.x == a.cnt_slot) ? 1 : 0;
+    if (threadIdx.x <= naggs) {
+        const int src = (threadIdx.x == naggs || threadIdx.x == cnt_slot) ? 1 : 0;
         out[threadIdx.x] = s_raw2[src];
     }
+}
+
+template <int MODE, typename PT, typename DT>
+__global__ void __launch_bounds__(FJ_THREADS, 4) k_pipe_fkjs(const __grid_constant__ FkjsArgs a,
+                                                             Slot16* __restrict__ parts,
+                                                             unsigned int* __restrict__ done,
+                                                             Slot16* __restrict__ out) {
+    const PT* __restrict__ pv = static_cast<const PT*>(a.pv);
+    const DT* __restrict__ dim = static_cast<const DT*>(a.dim);
+    const int64_t nthr = (int64_t)gridDim.x * FJ_THREADS;
+    const int64_t tid = (int64_t)blockIdx.x * FJ_THREADS + threadIdx.x;
+    int64_t sum = 0, cnt = 0;
+    // warp-uniform trip count (the __syncwarp below): lanes past n run with in = false
+    for (int64_t base = tid; base - (threadIdx.x & 31) < a.n; base += nthr * FJ_R) {
+        int64_t p[FJ_R];
+        bool q[FJ_R], ok[FJ_R];
+#pragma unroll
+        for (int k = 0; k < FJ_R; ++k) {
+            const int64_t r = base + k * nthr;
+            const bool in = r < a.n;
+            const int32_t f = in ? __ldcs(a.fk + r) : INT32_MIN;
+            const int64_t x = in ? (int64_t)__ldcs(pv + r) : (int64_t)Eps<PT>::value();
+            q[k] = in && x >= a.lo && x <= a.hi;
+            p[k] = (int64_t)f - a.bias;
+            ok[k] = f != INT32_MIN && p[k] >= 0 && p[k] < a.dim_len;  // else the gather gives epsilon
+            if (MODE == 2 && !q[k]) { p[k] = 0; ok[k] = a.dim_len > 0; }
+        }
+        DT g[FJ_R];
+        {
+            static_assert(FJ_R == 8, "one block of eight gathers");
+            const DT* ptr[8];
+            bool load[8];
+#pragma unroll
+            for (int k = 0; k < 8; ++k) {
+                load[k] = MODE == 0 ? (q[k] && ok[k]) : ok[k];
+                ptr[k] = dim + (load[k] ? p[k] : 0);
+            }
+            gather8(ptr, load, Eps<DT>::value(), g);
+        }
+        __syncwarp();  // all eight gathers issued before the first use
+#pragma unroll
+        for (int k = 0; k < FJ_R; ++k) {
+            const int64_t v = Eps<DT>::is(g[k]) ? 0 : (int64_t)g[k];  // an epsilon input adds nothing (A5)
+            if (MODE == 0) {
+                if (q[k]) { sum += v; cnt += 1; }
+            } else {
+                const int64_t pm = q[k] ? 1 : 0;
+                sum += v * pm;
+                cnt += pm;
+            }
+        }
+    }
+    scalar2_finish(sum, cnt, parts, done, out, a.naggs, a.cnt_slot);
+}
+
+// TMA variant of the Fig 16 fragment: fk and the predicate column stream
+// through a bulk-copy ring (producer warp), FJT_CW consumer warps evaluate
+// the predicate from shared memory and keep RPT gathers in flight per thread.
+constexpr int FJT_CW = 16;  // consumer warps
+constexpr int FJT_NT = FJT_CW * 32;
+constexpr int FJT_THREADS = FJT_NT + 32;
+constexpr int FJT_TILE = FJT_NT * 16;  // 16 gathers in flight per thread
+
+template <int MODE, typename PT, typename DT>
+__global__ void __launch_bounds__(FJT_THREADS, 1) k_pipe_fkjs_tma(const __grid_constant__ FkjsArgs a, int nstages,
+                                                                  int64_t ntiles, Slot16* __restrict__ parts,
+                                                                  unsigned int* __restrict__ done,
+                                                                  Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    constexpr int SB = FJT_TILE * (4 + (int)sizeof(PT));
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)nstages * SB);
+    uint64_t* empty = full + nstages;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const PT* __restrict__ pv = static_cast<const PT*>(a.pv);
+    const DT* __restrict__ dim = static_cast<const DT*>(a.dim);
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < nstages; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], FJT_CW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    int64_t sum = 0, cnt = 0;
+    constexpr int RPT = FJT_TILE / FJT_NT;
+    // RPT rows of one thread: predicate, then all gathers, then the fold
+    auto rows = [&](const int32_t* f, const int64_t* x, const bool* in) {
+        int64_t p[RPT];
+        bool q[RPT], ok[RPT];
+#pragma unroll
+        for (int k = 0; k < RPT; ++k) {
+            q[k] = in[k] && x[k] >= a.lo && x[k] <= a.hi;
+            p[k] = (int64_t)f[k] - a.bias;
+            ok[k] = f[k] != INT32_MIN && p[k] >= 0 && p[k] < a.dim_len;
+            if (MODE == 2 && !q[k]) { p[k] = 0; ok[k] = a.dim_len > 0; }
+        }
+        if (MODE == 0) {
+            bool any = false;
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) any |= q[k];
+            if (!__any_sync(VD_FULL, any)) return;  // no qualifying row in the warp: no gather, nothing to fold
+        }
+        DT g[RPT];
+        static_assert(RPT % 8 == 0, "gathers are issued in blocks of eight");
+#pragma unroll
+        for (int k0 = 0; k0 < RPT; k0 += 8) {
+            const DT* ptr[8];
+            bool load[8];
+#pragma unroll
+            for (int k = 0; k < 8; ++k) {
+                load[k] = MODE == 0 ? (q[k0 + k] && ok[k0 + k]) : (in[k0 + k] && ok[k0 + k]);
+                ptr[k] = dim + (load[k] ? p[k0 + k] : 0);
+            }
+            gather8(ptr, load, Eps<DT>::value(), g + k0);
+        }
+        __syncwarp();  // loads cannot sink past this point: all RPT are issued before the first use
+#pragma unroll
+        for (int k = 0; k < RPT; ++k) {
+            const int64_t v = Eps<DT>::is(g[k]) ? 0 : (int64_t)g[k];
+            if (MODE == 0) {
+                if (q[k]) { sum += v; cnt += 1; }
+            } else {
+                const int64_t pm = q[k] ? 1 : 0;
+                sum += v * pm;
+                cnt += pm;
+            }
+        }
+    };
+    if (warp == FJT_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % nstages);
+                if (it >= nstages) mbar_wait(&empty[s], (uint32_t)(((it / nstages) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * SB;
+                const int64_t r0 = tile * FJT_TILE;
+                mbar_expect_tx(&full[s], SB);
+                tma_load_1d(st, a.fk + r0, FJT_TILE * 4, &full[s], pol);
+                tma_load_1d(st + FJT_TILE * 4, pv + r0, FJT_TILE * (int)sizeof(PT), &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % nstages);
+            mbar_wait(&full[s], (uint32_t)((it / nstages) & 1));
+            const uint8_t* st = smem + (size_t)s * SB;
+            int32_t f[RPT];
+            int64_t x[RPT];
+            bool in[RPT];
+#pragma unroll
+            for (int k = 0; k < RPT; ++k) {
+                const int r = threadIdx.x + k * FJT_NT;
+                f[k] = reinterpret_cast<const int32_t*>(st)[r];
+                const PT xv = reinterpret_cast<const PT*>(st + FJT_TILE * 4)[r];
+                x[k] = Eps<PT>::is(xv) ? INT64_MIN : (int64_t)xv;  // lo > INT64_MIN: epsilon never qualifies
+                in[k] = true;
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+            rows(f, x, in);
+        }
+        if (blockIdx.x == 0) {  // ragged tail (< one tile)
+            for (int64_t base = ntiles * FJT_TILE + threadIdx.x; base - lane < a.n; base += (int64_t)FJT_NT * RPT) {
+                int32_t f[RPT];
+                int64_t x[RPT];
+                bool in[RPT];
+#pragma unroll
+                for (int k = 0; k < RPT; ++k) {
+                    const int64_t r = base + (int64_t)k * FJT_NT;
+                    in[k] = r < a.n;
+                    f[k] = in[k] ? a.fk[r] : INT32_MIN;
+                    const PT xv = in[k] ? pv[r] : Eps<PT>::value();
+                    x[k] = Eps<PT>::is(xv) ? INT64_MIN : (int64_t)xv;
+                }
+                rows(f, x, in);
+            }
+        }
+    }
+    __syncthreads();
+    scalar2_finish(sum, cnt, parts, done, out, a.naggs, a.cnt_slot);
 }
 
 // ============================================================================
@@ -2363,7 +2662,7 @@ static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols,
     A.ngroups = (int32_t)p->ngroups;
     A.n = n;
     constexpr size_t SB = FKG_TILE * 24;
-    const size_t fixed = (size_t)FKG_CW * p->ngroups * 16 + FKG_CW * 32 * 8 + (size_t)((A.ydays + 7) & ~7) * 2 +
+    const size_t fixed = (size_t)FKG_CW * 3 * (((size_t)p->ngroups + 32) & ~(size_t)31) * 4 + FKG_CW * 32 * 8 + (size_t)((A.ydays + 7) & ~7) * 2 +
                          2 * GF_MAXSTAGES * 8;
     const size_t budget = 200 * 1024;
     if (fixed + 2 * SB > budget) return VD_OK;
@@ -2374,17 +2673,131 @@ static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols,
     Slot16* parts = (Slot16*)((char*)ws + 256);
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-    if (narrow) {
-        cudaFuncSetAttribute(k_pipe_fkg<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_fkg<true><<<grid, FKG_THREADS, smem, s>>>(A, n / FKG_TILE, parts, dn, (Slot16*)out);
-    } else {
-        cudaFuncSetAttribute(k_pipe_fkg<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_fkg<false><<<grid, FKG_THREADS, smem, s>>>(A, n / FKG_TILE, parts, dn, (Slot16*)out);
-    }
+    // group-slot update: shared-memory atomics (default) or match_any leaders
+    const char* agg = getenv("VD_FKG_AGG");
+    const bool atom = !(agg && strcmp(agg, "match") == 0);
+    auto go = [&](auto kern) {
+        cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        kern<<<grid, FKG_THREADS, smem, s>>>(A, n / FKG_TILE, parts, dn, (Slot16*)out);
+    };
+    const char* pv_ = getenv("VD_FKG_PIPE");
+    const bool pipe = pv_ && strcmp(pv_, "1") == 0;
+    if (narrow && atom) pipe ? go(k_pipe_fkg<true, true, true>) : go(k_pipe_fkg<true, true, false>);
+    else if (narrow) pipe ? go(k_pipe_fkg<true, false, true>) : go(k_pipe_fkg<true, false, false>);
+    else if (atom) pipe ? go(k_pipe_fkg<false, true, true>) : go(k_pipe_fkg<false, true, false>);
+    else pipe ? go(k_pipe_fkg<false, false, true>) : go(k_pipe_fkg<false, false, false>);
     ++*nl;
     e = cudaGetLastError();
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     set_fragment("fk_group");
+    *done = true;
+    return VD_OK;
+}
+
+// ---- selective FK join (Fig 16) matching -----------------------------------------------
+template <int MODE, typename PT, typename DT>
+static void launch_fkjs_tma1(const FkjsArgs& A, int64_t n, Slot16* parts, unsigned* dn, Slot16* out, cudaStream_t s) {
+    constexpr size_t SB = FJT_TILE * (4 + sizeof(PT));
+    const int nstages = (int)std::min<size_t>(8, (200 * 1024) / SB);
+    const size_t smem = (size_t)nstages * SB + 2 * nstages * 8;
+    cudaFuncSetAttribute(k_pipe_fkjs_tma<MODE, PT, DT>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    k_pipe_fkjs_tma<MODE, PT, DT><<<num_sms(), FJT_THREADS, smem, s>>>(A, nstages, n / FJT_TILE, parts, dn, out);
+}
+
+template <int MODE>
+static void launch_fkjs_tma(const FkjsArgs& A, int pdt, int ddt, int64_t n, Slot16* parts, unsigned* dn, Slot16* out,
+                            cudaStream_t s) {
+    if (pdt == VD_I32 && ddt == VD_I64) launch_fkjs_tma1<MODE, int32_t, int64_t>(A, n, parts, dn, out, s);
+    else if (pdt == VD_I32) launch_fkjs_tma1<MODE, int32_t, int32_t>(A, n, parts, dn, out, s);
+    else if (ddt == VD_I64) launch_fkjs_tma1<MODE, int64_t, int64_t>(A, n, parts, dn, out, s);
+    else launch_fkjs_tma1<MODE, int64_t, int32_t>(A, n, parts, dn, out, s);
+}
+
+template <int MODE>
+static void launch_fkjs(const FkjsArgs& A, int pdt, int ddt, int grid, Slot16* parts, unsigned* dn, Slot16* out,
+                        cudaStream_t s) {
+    if (pdt == VD_I32 && ddt == VD_I64) k_pipe_fkjs<MODE, int32_t, int64_t><<<grid, FJ_THREADS, 0, s>>>(A, parts, dn, out);
+    else if (pdt == VD_I32) k_pipe_fkjs<MODE, int32_t, int32_t><<<grid, FJ_THREADS, 0, s>>>(A, parts, dn, out);
+    else if (ddt == VD_I64) k_pipe_fkjs<MODE, int64_t, int64_t><<<grid, FJ_THREADS, 0, s>>>(A, parts, dn, out);
+    else k_pipe_fkjs<MODE, int64_t, int32_t><<<grid, FJ_THREADS, 0, s>>>(A, parts, dn, out);
+}
+
+static vd_status try_fkjs(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                          void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
+    *done = false;
+    const char* var = getenv("VD_FKJS_VARIANT");
+    if (var && strcmp(var, "off") == 0) return VD_OK;
+    if (p->nkeyparts != 0 || p->ngroups != 1 || p->ngathers != 1 || p->pred.nconj != 1) return VD_OK;
+    const int fkc = p->gathers[0].fk_col;
+    if (fkc >= ncols || cols[fkc].dtype != VD_I32) return VD_OK;
+    const vd_column& dim = dims[p->gathers[0].dim_col];
+    if (dim.dtype != VD_I32 && dim.dtype != VD_I64) return VD_OK;
+    int pc = -1;
+    int64_t lo = INT64_MIN + 1, hi = INT64_MAX;
+    for (int t = 0; t < p->pred.conj[0].nterms; ++t) {
+        const vd_term& tm = p->pred.conj[0].terms[t];
+        if (tm.col >= ncols || (pc >= 0 && tm.col != pc)) return VD_OK;
+        pc = tm.col;
+        if (!term_interval(tm, &lo, &hi)) return VD_OK;
+    }
+    if (pc < 0 || (cols[pc].dtype != VD_I32 && cols[pc].dtype != VD_I64)) return VD_OK;
+    if (cols[pc].dtype == VD_I32) lo = std::max<int64_t>(lo, (int64_t)INT32_MIN + 1);
+    FkjsArgs A;
+    std::memset(&A, 0, sizeof(A));
+    A.sum_slot = A.cnt_slot = -1;
+    A.naggs = p->naggs;
+    for (int g = 0; g < p->naggs; ++g) {
+        const vd_agg& ag = p->aggs[g];
+        if (ag.kind == VD_AGG_COUNT) { if (A.cnt_slot >= 0) return VD_OK; A.cnt_slot = g; continue; }
+        if (ag.kind != VD_AGG_SUM || A.sum_slot >= 0 || ag.nfactors != 1 || !plain_col(ag.f[0]) ||
+            ag.f[0].col != ncols)
+            return VD_OK;
+        A.sum_slot = g;
+    }
+    if (A.sum_slot < 0) return VD_OK;
+    const Bound bd = col_bound(p, cols, ncols, dims, ncols);
+    if (!bd.known) return VD_OK;
+    const int grid = num_sms() * 4;
+    // both variants: at least num_sms() * FKG_NT threads, plus a ragged tail
+    const double rows_per_thread = std::ceil((double)n / ((double)num_sms() * FKG_NT)) + 2.0 * FJT_TILE / FJT_NT;
+    if (std::max(std::fabs(bd.lo), std::fabs(bd.hi)) * rows_per_thread * 32.0 >= 9.0e18) return VD_OK;
+    A.fk = (const int32_t*)cols[fkc].data;
+    A.pv = cols[pc].data;
+    A.dim = dim.data;
+    A.n = n;
+    A.dim_len = dim.len;
+    A.bias = p->gathers[0].bias;
+    A.lo = lo;
+    A.hi = hi;
+    unsigned int* dn = (unsigned int*)ws;
+    Slot16* parts = (Slot16*)((char*)ws + 256);
+    cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    // Branching reads the dimension only for qualifying rows: the TMA ring
+    // streams the two columns at full bandwidth (2.5x the plain loads at low
+    // selectivity).  The predicated strategies gather every row and are bound
+    // by random DRAM accesses, where the plain-load kernel (more warps, fewer
+    // LSU stalls) is faster.  VD_FKJS_VARIANT=ldg|tma overrides; TMA needs
+    // 16-byte aligned columns.
+    bool tma = p->sel_mode == VD_SEL_BRANCH;
+    if (var && strcmp(var, "ldg") == 0) tma = false;
+    if (var && strcmp(var, "tma") == 0) tma = true;
+    tma = tma && ((uintptr_t)A.fk % 16) == 0 && ((uintptr_t)A.pv % 16) == 0;
+    const int pdt = cols[pc].dtype, ddt = dim.dtype;
+    Slot16* o = (Slot16*)out;
+    if (tma) {
+        if (p->sel_mode == VD_SEL_BRANCH) launch_fkjs_tma<0>(A, pdt, ddt, n, parts, dn, o, s);
+        else if (p->sel_mode == VD_SEL_PREDICATED) launch_fkjs_tma<1>(A, pdt, ddt, n, parts, dn, o, s);
+        else launch_fkjs_tma<2>(A, pdt, ddt, n, parts, dn, o, s);
+    } else {
+        if (p->sel_mode == VD_SEL_BRANCH) launch_fkjs<0>(A, pdt, ddt, grid, parts, dn, o, s);
+        else if (p->sel_mode == VD_SEL_PREDICATED) launch_fkjs<1>(A, pdt, ddt, grid, parts, dn, o, s);
+        else launch_fkjs<2>(A, pdt, ddt, grid, parts, dn, o, s);
+    }
+    ++*nl;
+    e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    set_fragment("fk_select_sum");
     *done = true;
     return VD_OK;
 }
@@ -2830,6 +3243,8 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_fkg(p, cols, ncols, n, dims, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
+        st = try_fkjs(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_star(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;

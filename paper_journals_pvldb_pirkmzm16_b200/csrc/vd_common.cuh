@@ -67,6 +67,21 @@ __device__ __forceinline__ int ld_stream4(const void* p) {
 }
 
 // ---- gpu-scope acquire/release on 64-bit status words ---------------------
+// Eight predicated read-only gathers (default value where !pred) in one
+// inline-PTX block: every address is ready before the first load issues, so
+// all eight are in flight together (left to itself the compiler consumes each
+// gather before computing the next address).
+__device__ __forceinline__ void gather8(const int64_t* const* p, const bool* pr, int64_t dflt, int64_t* v) {
+    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b64 %0, %24;\n\tmov.b64 %1, %24;\n\tmov.b64 %2, %24;\n\tmov.b64 %3, %24;\n\tmov.b64 %4, %24;\n\tmov.b64 %5, %24;\n\tmov.b64 %6, %24;\n\tmov.b64 %7, %24;\n\t@q0 ld.global.nc.b64 %0, [%8];\n\t@q1 ld.global.nc.b64 %1, [%9];\n\t@q2 ld.global.nc.b64 %2, [%10];\n\t@q3 ld.global.nc.b64 %3, [%11];\n\t@q4 ld.global.nc.b64 %4, [%12];\n\t@q5 ld.global.nc.b64 %5, [%13];\n\t@q6 ld.global.nc.b64 %6, [%14];\n\t@q7 ld.global.nc.b64 %7, [%15];\n\t}"
+                 : "=l"(v[0]), "=l"(v[1]), "=l"(v[2]), "=l"(v[3]), "=l"(v[4]), "=l"(v[5]), "=l"(v[6]), "=l"(v[7])
+                 : "l"(p[0]), "l"(p[1]), "l"(p[2]), "l"(p[3]), "l"(p[4]), "l"(p[5]), "l"(p[6]), "l"(p[7]), "r"((int)pr[0]), "r"((int)pr[1]), "r"((int)pr[2]), "r"((int)pr[3]), "r"((int)pr[4]), "r"((int)pr[5]), "r"((int)pr[6]), "r"((int)pr[7]), "l"(dflt));
+}
+__device__ __forceinline__ void gather8(const int32_t* const* p, const bool* pr, int32_t dflt, int32_t* v) {
+    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b32 %0, %24;\n\tmov.b32 %1, %24;\n\tmov.b32 %2, %24;\n\tmov.b32 %3, %24;\n\tmov.b32 %4, %24;\n\tmov.b32 %5, %24;\n\tmov.b32 %6, %24;\n\tmov.b32 %7, %24;\n\t@q0 ld.global.nc.b32 %0, [%8];\n\t@q1 ld.global.nc.b32 %1, [%9];\n\t@q2 ld.global.nc.b32 %2, [%10];\n\t@q3 ld.global.nc.b32 %3, [%11];\n\t@q4 ld.global.nc.b32 %4, [%12];\n\t@q5 ld.global.nc.b32 %5, [%13];\n\t@q6 ld.global.nc.b32 %6, [%14];\n\t@q7 ld.global.nc.b32 %7, [%15];\n\t}"
+                 : "=r"(v[0]), "=r"(v[1]), "=r"(v[2]), "=r"(v[3]), "=r"(v[4]), "=r"(v[5]), "=r"(v[6]), "=r"(v[7])
+                 : "l"(p[0]), "l"(p[1]), "l"(p[2]), "l"(p[3]), "l"(p[4]), "l"(p[5]), "l"(p[6]), "l"(p[7]), "r"((int)pr[0]), "r"((int)pr[1]), "r"((int)pr[2]), "r"((int)pr[3]), "r"((int)pr[4]), "r"((int)pr[5]), "r"((int)pr[6]), "r"((int)pr[7]), "r"(dflt));
+}
+
 __device__ __forceinline__ uint64_t ld_acquire_u64(const uint64_t* p) {
     uint64_t v;
     asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(v) : "l"(p) : "memory");

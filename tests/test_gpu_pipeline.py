@@ -402,17 +402,22 @@ def test_fkj_q9_gather_fold_fragment(variant):
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
+@pytest.mark.parametrize("variant", ["fk_select_sum_tma", "fk_select_sum_ldg", "gather_fold"])
 @pytest.mark.parametrize("mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED, vd.VD_SEL_PREDICATED_LOOKUP])
 @pytest.mark.parametrize("sel", [0.0, 0.013, 0.5, 1.0])
-def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel):
+def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel, variant):
     """Fig 16: branching, predicated aggregation and predicated
     lookups give the same SUM(target.v) and count as the oracle's program
-    Gather(target.v, fk - 1) -> FoldSelect(v < t) -> FoldSum."""
+    Gather(target.v, fk - 1) -> FoldSelect(v < t) -> FoldSum, with epsilon in
+    every column and foreign keys outside the target (gathered as epsilon)."""
+    import os
     n, m = 100003, 5000
     rng = np.random.default_rng(7)
-    fk = rng.integers(1, m + 1, n).astype(np.int32)
+    fk = rng.integers(-1, m + 3, n).astype(np.int32)
     v = rng.integers(0, plans.FKJSEL_VMAX, n).astype(np.int32)
     tv = rng.integers(-10**6, 10**6, m).astype(np.int64)
+    efk, ev, et = rng.random(n) < 0.01, rng.random(n) < 0.01, rng.random(m) < 0.01
+    fk[efk], v[ev], tv[et] = -2**31, -2**31, -2**63
     thr = int(round(sel * plans.FKJSEL_VMAX))
     prog = f"""
     p := Subtract(fact.fk, 1)
@@ -421,15 +426,20 @@ def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel):
     pos := FoldSelect(q)
     sel := Gather(g, pos)
     s := FoldSum(sel)
-    c := FoldCount(sel)
+    c := FoldCount(pos)
     """
-    po = oracle.run(prog, fact__fk=fk, fact__v=v, target__v=tv)
+    po = oracle.run(prog, fact__fk=(fk, efk), fact__v=(v, ev), target__v=(tv, et))
     exp_s, exp_c = po.get("s")[0], po.get("c")[0]
     keep, views = load([fk, v])
     dkeep, dviews = load([tv])
     plan = plans.fkjsel(thr, mode)
-    got = vd.decode_partials(run(plan, views, n, dviews, want=("gather_fold",))[0], plan)
-    if exp_c == 0:
+    os.environ["VD_FKJS_VARIANT"] = {"gather_fold": "off", "fk_select_sum_ldg": "ldg", "fk_select_sum_tma": "tma"}[variant]
+    try:
+        got = vd.decode_partials(run(plan, views, n, dviews, want=(variant.replace("_ldg", "").replace("_tma", ""),))[0],
+                                 plan)
+    finally:
+        os.environ.pop("VD_FKJS_VARIANT", None)
+    if not exp_c:
         assert got == {}
     else:
-        assert got == {0: [exp_s, exp_c, exp_c]}
+        assert got == {0: [exp_s or 0, exp_c, exp_c]}
