@@ -45,7 +45,7 @@ def parse():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
     ap.add_argument("--workload", default="q1",
-                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused"])
+                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14"])
     ap.add_argument("--chunk", type=int, default=0,
                     help="select_unfused: rows per materialised chunk (0 = whole table; Fig 15 'Vectorized')")
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
@@ -53,6 +53,10 @@ def parse():
     ap.add_argument("--selectivity", type=float, default=0.5, help="select workload: fraction selected")
     ap.add_argument("--rows", type=int, default=None, help="select workload: rows (default 1e9)")
     ap.add_argument("--generic", action="store_true", help="force the generic fragment")
+    ap.add_argument("--strategy", default="layout", choices=["single", "separate", "layout"],
+                    help="fig14: Single Loop / Separate Loops / Layout Transform (P:L1156-1193)")
+    ap.add_argument("--pattern", default="random", choices=["random", "sequential"], help="fig14 lookup pattern")
+    ap.add_argument("--target-mb", type=int, default=128, help="fig14 target table size (two int32 columns)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
@@ -64,7 +68,7 @@ def parse():
 
 def default_sf(w):
     return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0,
-            "select_unfused": 0.0}[w]
+            "select_unfused": 0.0, "fig14": 0.0}[w]
 
 
 # ---------------------------------------------------------------------------
@@ -207,6 +211,8 @@ def main():
         return selpos_main(args, rank, world, local)
     if args.workload == "select_unfused":
         return unfused_main(args, rank, world, local)
+    if args.workload == "fig14":
+        return fig14_main(args, rank, world, local)
 
     import torch
     import torch.distributed as dist
@@ -382,7 +388,8 @@ def main():
         "hbm_gbs": achieved,
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                      "frac": achieved / peak, "peak_kind": peak_kind,
-                     "traffic": ncu_traffic(w), "bytes_per_row": bpr,
+                     "traffic": ncu_traffic(f"fkjsel_s{args.selectivity:g}_{args.sel_mode}" if w == "fkjsel" else w),
+                     "bytes_per_row": bpr,
                      "kernel": "k_pipe_q1+k_q1_remap" if w == "q1" and not args.generic else "vd_run_pipeline",
                      "kernel_ms": kernel_ms},
         "clocks": clk,
@@ -462,7 +469,8 @@ def selpos_main(args, rank, world, local):
                        "selected": c, "achieved_selectivity": c / n,
                        "l2": f"input {4 * n / 1e9:.1f} GB > 126 MB L2: no flush needed"},
             "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
-                         "peak_kind": kind, "traffic": None, "kernel": "k_select", "kernel_ms": ms},
+                         "peak_kind": kind, "traffic": ncu_traffic(f"selpos_s{args.selectivity:g}_{args.sel_mode}"),
+                         "kernel": "k_select", "kernel_ms": ms},
             "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
     if rank == 0:
         print(json.dumps(line), flush=True)
@@ -580,6 +588,91 @@ def unfused_main(args, rank, world, local):
                          "peak_kind": kind, "traffic": None, "kernel": "select+gather+fold (unfused)",
                          "kernel_ms": ms},
             "result": float(total.item()), "e2e": None}
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    comm.close()
+
+
+def fig14_main(args, rank, world, local):
+    """Multi-column FK lookups (Fig 14): n positions resolved
+    into the two int32 columns of a target table of --target-mb, by a Single
+    Loop (vd_gather_multi), Separate Loops (one vd_gather per column), or a
+    Layout Transform (vd_zip of the target into 8-byte rows, inside the timed
+    step, then vd_gather_rows).  Lookups are sequential (i mod m) or uniform
+    random.  Algorithmic bytes per position: 4 (pos) + 2 x 4 gathered + 2 x 4
+    written = 20 B."""
+    import torch
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % ndev)
+    dev = torch.device("cuda", local % ndev)
+    comm = Comm(world, args.dist_backend, dev)
+    stream = torch.cuda.current_stream()
+    n_total = args.rows or 200_000_000
+    a, b = rank * n_total // world, (rank + 1) * n_total // world
+    n = b - a
+    m = args.target_mb * (1 << 20) // 8
+    t0 = torch.empty(m, dtype=torch.int32, device=dev)
+    t1 = torch.empty(m, dtype=torch.int32, device=dev)
+    gen.device(gen.I32_UNIFORM, t0.data_ptr(), m, 0, seed=args.seed + 3, p0=0, p1=10**9, stream=stream.cuda_stream)
+    gen.device(gen.I32_UNIFORM, t1.data_ptr(), m, 0, seed=args.seed + 4, p0=0, p1=10**9, stream=stream.cuda_stream)
+    pos = torch.empty(n, dtype=torch.int32, device=dev)
+    if args.pattern == "random":
+        gen.device(gen.I32_UNIFORM, pos.data_ptr(), n, a, seed=args.seed + 5, p0=0, p1=m - 1, stream=stream.cuda_stream)
+    else:
+        torch.remainder(torch.arange(a, b, device=dev, dtype=torch.int64), m, out=pos)
+    o0 = torch.empty(n, dtype=torch.int32, device=dev)
+    o1 = torch.empty(n, dtype=torch.int32, device=dev)
+    cols = [vd.column(t0), vd.column(t1)]
+    dts = [vd.VD_I32, vd.VD_I32]
+    _, stride = vd.row_layout(dts)
+    rows = torch.empty(m * stride, dtype=torch.uint8, device=dev)
+    launches = {"single": 1, "separate": 2, "layout": 2}[args.strategy]
+
+    def step():
+        if args.strategy == "single":
+            vd.gather_multi(cols, pos, n, 0, [o0, o1], stream=stream)
+        elif args.strategy == "separate":
+            vd.gather(cols[0], pos, n, 0, o0, stream=stream)
+            vd.gather(cols[1], pos, n, 0, o1, stream=stream)
+        else:
+            vd.zip_rows(cols, rows, stream=stream)
+            vd.gather_rows(rows, m, dts, pos, n, 0, [o0, o1], stream=stream)
+
+    for _ in range(max(args.warmup, 3)):
+        step()
+    torch.cuda.synchronize()
+    ok = bool(torch.equal(o0, t0[pos.long()])) and bool(torch.equal(o1, t1[pos.long()]))
+    steps = args.steps or 50
+    clocks = ClockSampler(local)
+    clocks.start()
+    time.sleep(0.3)
+    comm.barrier()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    clk = clocks.stop()
+    ms = comm.max([e0.elapsed_time(e1) / steps])[0]
+    peak, kind = hbm_peak()
+    alg = 20 * n / (ms * 1e-3) / 1e9
+    line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "int32", "data": "synthetic (uniform int32 target, gen/vd_gen.h)",
+            "config": {"workload": f"fig14_{args.strategy}_{args.pattern}_{args.target_mb}MB_{n_total}",
+                       "strategy": args.strategy, "pattern": args.pattern, "target_mb": args.target_mb,
+                       "positions": n_total, "l2": "positions + outputs 2.4 GB per step > 126 MB L2"},
+            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
+                         "peak_kind": kind, "traffic": None, "bytes_per_row": 20,
+                         "kernel": {"single": "k_gather", "separate": "k_gather x2",
+                                    "layout": "k_zip + k_gather_rows"}[args.strategy], "kernel_ms": ms},
+            "clocks": clk, "e2e": None, "gpu_launches": launches * steps, "result_ok": ok}
     if rank == 0:
         print(json.dumps(line), flush=True)
     comm.close()

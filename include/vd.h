@@ -244,6 +244,30 @@ vd_status vd_gather(const vd_column* src, const int32_t* pos, int64_t n, int64_t
 vd_status vd_gather_multi(const vd_column* srcs, int32_t nsrc, const int32_t* pos, int64_t n, int64_t bias,
                           void* const* outs_host, void* stream);
 
+/* Just-in-time layout transformation (Fig 14 "Layout Transform",
+ * P:L1156-1193): Zip + materialise the target columns into row-wise storage
+ * (P:L1185-1188), then resolve positions with one lookup per row.
+ *
+ * vd_row_layout (host only, no device work): the row format shared by
+ * vd_zip and vd_gather_rows.  Field k (dtypes[k], 1 <= nfields <= 4) sits at
+ * offsets[k] bytes, each field aligned to its own size, in declaration
+ * order; *stride = the packed size rounded up to a power of two >= 8, so a
+ * row never straddles a 32-byte sector.  VD_E_UNSUPPORTED if the packed
+ * size exceeds 32 bytes.
+ *
+ * vd_zip: rows[i] (stride bytes at out_rows + i*stride) = the fields
+ * cols[0..ncols)[i]; every column has cols[0].len rows; out_bytes >=
+ * len*stride; padding bytes are zero; epsilon values are copied as is.
+ *
+ * vd_gather_rows: for i in [0, n), p = pos[i] - bias: outs_host[k][i] =
+ * field k of row p (dtype dtypes[k]); a negative (epsilon) or out-of-bounds
+ * position gives epsilon in every field (reading A11).  outs_host is a host
+ * array of nfields device pointers. */
+vd_status vd_row_layout(const int32_t* dtypes, int32_t nfields, int32_t* offsets, int32_t* stride);
+vd_status vd_zip(const vd_column* cols, int32_t ncols, void* out_rows, int64_t out_bytes, void* stream);
+vd_status vd_gather_rows(const void* rows, int64_t nrows, const int32_t* dtypes, int32_t nfields, const int32_t* pos,
+                         int64_t n, int64_t bias, void* const* outs_host, void* stream);
+
 /* ---------------------------------------------------------------------- */
 /* a5  Scatter / Partition (Table 2; §3.1.3)        */
 /* ---------------------------------------------------------------------- */

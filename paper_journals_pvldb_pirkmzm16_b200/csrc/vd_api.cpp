@@ -439,6 +439,61 @@ vd_status vd_gather(const vd_column* src, const int32_t* pos, int64_t n, int64_t
     return vd_gather_multi(src, 1, pos, n, bias, outs, stream);
 }
 
+vd_status vd_row_layout(const int32_t* dtypes, int32_t nfields, int32_t* offsets, int32_t* stride) {
+    if (!dtypes || !offsets || !stride) return VD_E_NULL;
+    if (nfields < 1 || nfields > VD_MAX_GATHERS) { set_error("row layout: 1..4 fields"); return VD_E_ARG; }
+    for (int k = 0; k < nfields; ++k)
+        if (!valid_dtype(dtypes[k])) { set_error("row layout: bad dtype"); return VD_E_DTYPE; }
+    if (!row_layout(dtypes, nfields, offsets, stride)) {
+        set_error("row layout: a row must fit 32 bytes");
+        return VD_E_UNSUPPORTED;
+    }
+    return VD_OK;
+}
+
+vd_status vd_zip(const vd_column* cols, int32_t ncols, void* out_rows, int64_t out_bytes, void* stream) {
+    reset_launches();
+    if (!cols) return VD_E_NULL;
+    if (ncols < 1 || ncols > VD_MAX_GATHERS) { set_error("zip: 1..4 columns"); return VD_E_ARG; }
+    int32_t dts[VD_MAX_GATHERS], offs[VD_MAX_GATHERS], stride;
+    for (int k = 0; k < ncols; ++k) {
+        vd_status st = check_col(&cols[k], cols[0].len, "zip");
+        if (st != VD_OK) return st;
+        dts[k] = cols[k].dtype;
+    }
+    vd_status st = vd_row_layout(dts, ncols, offs, &stride);
+    if (st != VD_OK) return st;
+    if (out_bytes < cols[0].len * (int64_t)stride) { set_error("zip: output smaller than len * stride"); return VD_E_SHAPE; }
+    if (cols[0].len > 0 && !out_rows) return VD_E_NULL;
+    if (((uintptr_t)out_rows % 16) != 0) { set_error("zip: rows must be 16-byte aligned"); return VD_E_ARG; }
+    st = check_device();
+    if (st != VD_OK) return st;
+    int nl = 0;
+    st = cuda_status(launch_zip(cols, ncols, out_rows, (cudaStream_t)stream, &nl));
+    count_launches(nl);
+    return st;
+}
+
+vd_status vd_gather_rows(const void* rows, int64_t nrows, const int32_t* dtypes, int32_t nfields, const int32_t* pos,
+                         int64_t n, int64_t bias, void* const* outs, void* stream) {
+    reset_launches();
+    int32_t offs[VD_MAX_GATHERS], stride;
+    vd_status st = vd_row_layout(dtypes, nfields, offs, &stride);
+    if (st != VD_OK) return st;
+    if (n < 0 || nrows < 0) return VD_E_SHAPE;
+    if (n > 0 && (!pos || !outs)) { set_error("gather_rows: NULL pos/outs"); return VD_E_NULL; }
+    if (nrows > 0 && !rows) return VD_E_NULL;
+    if (((uintptr_t)rows % 16) != 0) { set_error("gather_rows: rows must be 16-byte aligned"); return VD_E_ARG; }
+    for (int k = 0; k < nfields && n > 0; ++k)
+        if (!outs[k]) { set_error("gather_rows: NULL out"); return VD_E_NULL; }
+    st = check_device();
+    if (st != VD_OK) return st;
+    int nl = 0;
+    st = cuda_status(launch_gather_rows(rows, nrows, dtypes, nfields, pos, n, bias, outs, (cudaStream_t)stream, &nl));
+    count_launches(nl);
+    return st;
+}
+
 vd_status vd_scatter(const vd_column* src, const int32_t* pos, int64_t n, void* out, int64_t out_len, int32_t flags,
                      void* ws, size_t ws_bytes, void* stream) {
     reset_launches();

@@ -79,6 +79,10 @@ cudaError_t launch_fold(FoldOp op, const vd_column& vals, const CtrlInfo& ci, vo
 // k_gather.cu
 cudaError_t launch_gather(const vd_column* srcs, int nsrc, const int32_t* pos, int64_t n, int64_t bias,
                           void* const* outs, cudaStream_t s, int* nlaunch);
+bool row_layout(const int32_t* dtypes, int nfields, int32_t* offsets, int32_t* stride);
+cudaError_t launch_zip(const vd_column* cols, int ncols, void* out_rows, cudaStream_t s, int* nl);
+cudaError_t launch_gather_rows(const void* rows, int64_t nrows, const int32_t* dtypes, int nfields,
+                               const int32_t* pos, int64_t n, int64_t bias, void* const* outs, cudaStream_t s, int* nl);
 // k_scatter.cu
 size_t scatter_ws_bytes(int64_t out_len);
 cudaError_t launch_scatter(const vd_column& src, const int32_t* pos, int64_t n, void* out, int64_t out_len,

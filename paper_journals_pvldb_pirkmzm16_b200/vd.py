@@ -113,6 +113,10 @@ _sigs = {
                               c_void_p]),
     "vd_gather": (c_int32, [_P(vd_column), c_void_p, c_int64, c_int64, c_void_p, c_void_p]),
     "vd_gather_multi": (c_int32, [_P(vd_column), c_int32, c_void_p, c_int64, c_int64, _P(c_void_p), c_void_p]),
+    "vd_row_layout": (c_int32, [_P(c_int32), c_int32, _P(c_int32), _P(c_int32)]),
+    "vd_zip": (c_int32, [_P(vd_column), c_int32, c_void_p, c_int64, c_void_p]),
+    "vd_gather_rows": (c_int32, [c_void_p, c_int64, _P(c_int32), c_int32, c_void_p, c_int64, c_int64, _P(c_void_p),
+                                 c_void_p]),
     "vd_scatter": (c_int32, [_P(vd_column), c_void_p, c_int64, c_void_p, c_int64, c_int32, c_void_p, c_size_t,
                              c_void_p]),
     "vd_partition": (c_int32, [_P(vd_column), c_int64, c_int64, c_void_p, c_void_p, c_void_p, c_size_t, c_void_p]),
@@ -372,6 +376,31 @@ def gather_multi(srcs: Sequence[vd_column], pos, n, bias, outs, stream=None):
     arr = _cols_array(srcs)
     o = (c_void_p * len(outs))(*[t.data_ptr() for t in outs])
     _ok(_L.vd_gather_multi(arr, len(srcs), _ptr(pos), n, bias, o, _stream(stream)), "vd_gather_multi")
+
+
+def row_layout(dtypes: Sequence[int]):
+    """vd_row_layout: (field offsets, row stride) of the row-wise format (Fig 14 Layout Transform)."""
+    k = len(dtypes)
+    dt = (c_int32 * k)(*dtypes)
+    offs = (c_int32 * k)()
+    st = c_int32()
+    _ok(_L.vd_row_layout(dt, k, offs, ctypes.byref(st)), "vd_row_layout")
+    return list(offs), st.value
+
+
+def zip_rows(cols: Sequence[vd_column], out_rows, stream=None):
+    """vd_zip: materialise the columns row-wise into `out_rows` (CUDA uint8 tensor, len*stride bytes)."""
+    arr = _cols_array(cols)
+    _ok(_L.vd_zip(arr, len(cols), _ptr(out_rows), out_rows.numel() * out_rows.element_size(), _stream(stream)),
+        "vd_zip")
+
+
+def gather_rows(rows, nrows, dtypes: Sequence[int], pos, n, bias, outs, stream=None):
+    """vd_gather_rows: resolve positions into the row-wise table, field k -> outs[k]."""
+    k = len(dtypes)
+    dt = (c_int32 * k)(*dtypes)
+    o = (c_void_p * k)(*[t.data_ptr() for t in outs])
+    _ok(_L.vd_gather_rows(_ptr(rows), nrows, dt, k, _ptr(pos), n, bias, o, _stream(stream)), "vd_gather_rows")
 
 
 def scatter(src: vd_column, pos, n, out, out_len, unique=False, ws=None, stream=None):

@@ -4,6 +4,7 @@
   python scripts/sweep.py fig1  > gpurun_out/sweep_fig1.jsonl   # C2: 1e9 f32 -> positions
   python scripts/sweep.py fig15 > gpurun_out/sweep_fig15.jsonl  # selective aggregation (select + FoldSum)
   python scripts/sweep.py fig16 > gpurun_out/sweep_fig16.jsonl  # selective FK join: branch / predicated / lookup
+  python scripts/sweep.py fig14 > gpurun_out/sweep_fig14.jsonl  # multi-column lookups: single / separate / layout
 
 Fig 1 and Fig 15: branching vs
 predicated (cursor arithmetic) over selectivities 1..100 % (plus the Fig 15
@@ -45,10 +46,27 @@ def table(files):
               f"{d['value'] / 1e9:.1f} | {d['roofline']['achieved']:.0f} | {d['roofline']['frac']:.3f} |")
 
 
+def fig14():
+    """Fig 14: strategy x lookup pattern x target size."""
+    for pattern in ["sequential", "random"]:
+        for mb in [4, 128]:
+            for strat in ["single", "separate", "layout"]:
+                cmd = [sys.executable, os.path.join(ROOT, "bench.py"), "--workload", "fig14", "--strategy", strat,
+                       "--pattern", pattern, "--target-mb", str(mb), "--steps", "30"]
+                out = subprocess.run(cmd, capture_output=True, text=True, timeout=600)
+                line = out.stdout.strip().splitlines()[-1] if out.stdout.strip() else "{}"
+                d = json.loads(line)
+                d["_sel"] = f"{pattern} {mb}MB"
+                d["_mode"] = strat
+                print(json.dumps(d), flush=True)
+
+
 def main():
     what = sys.argv[1]
     if what == "table":
         return table(sys.argv[2:])
+    if what == "fig14":
+        return fig14()
     workload = {"fig1": "selpos", "fig15": "select", "fig16": "fkjsel"}[what]
     modes = ["branch", "predicated", "lookup"] if what == "fig16" else ["branch", "predicated"]
     for s in SEL:

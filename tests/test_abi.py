@@ -147,3 +147,26 @@ def test_pipeline_descriptor_round_trip():
     assert p.pred.conj[0].terms[0].cmp == vd.VD_CMP_LE and p.pred.conj[0].terms[0].ival == 10471
     q = vd.pred([[(0, "in", [0, 3, 63])]])
     assert q.conj[0].terms[0].ival == (1 | 8 | (1 << 63)) - (1 << 64)
+
+
+def test_row_layout_reading_fig14():
+    """vd_row_layout (host only): fields in order, each aligned to its size,
+    no overlap, stride a power of two >= 8 holding the packed row, rows of
+    more than 32 bytes refused (one sector per lookup)."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    size = {vd.VD_U8: 1, vd.VD_I32: 4, vd.VD_F32: 4, vd.VD_I64: 8, vd.VD_F64: 8}
+    import itertools
+    for k in range(1, 5):
+        for dts in itertools.product(list(size), repeat=k):
+            if sum(size[d] for d in dts) > 24:
+                continue
+            offs, stride = vd.row_layout(list(dts))
+            assert stride >= 8 and stride & (stride - 1) == 0 and stride <= 32
+            end = 0
+            for d, o in zip(dts, offs):
+                assert o % size[d] == 0 and o >= end
+                end = o + size[d]
+            assert end <= stride and stride // 2 < max(end, 5)
+    assert vd.row_layout([vd.VD_I32, vd.VD_I32]) == ([0, 4], 8)
+    with pytest.raises(vd.VdError):
+        vd.row_layout([vd.VD_U8, vd.VD_F64, vd.VD_F64, vd.VD_F64, vd.VD_U8])

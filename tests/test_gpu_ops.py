@@ -329,6 +329,58 @@ def test_gather_multi_vs_interpreter(n, bias):
             assert np.array_equal(got.astype(np.int64), exp)
 
 
+@pytest.mark.parametrize("fields", [("i32", "i32"), ("u8", "i64", "i32"), ("f32", "i64", "u8", "i32"),
+                                    ("i64", "i64", "i64", "i64"), ("f64",)])
+@pytest.mark.parametrize("n", [0, 1, 4097, 200003])
+def test_layout_transform_vs_interpreter(fields, n):
+    """Fig 14 Layout Transform: vd_zip materialises the target
+    columns row-wise, vd_gather_rows resolves positions into the rows; every
+    field equals the oracle's Gather(Zip(...), p) (epsilon in the columns,
+    negative and out-of-bounds positions give epsilon, reading A11)."""
+    rng = np.random.default_rng(n + len(fields))
+    m = 3001
+    gen_ = {"u8": lambda: rng.integers(0, 255, m).astype(np.uint8),
+            "i32": lambda: rng.integers(-10**9, 10**9, m).astype(np.int32),
+            "i64": lambda: rng.integers(-10**17, 10**17, m).astype(np.int64),
+            "f32": lambda: rng.random(m).astype(np.float32),
+            "f64": lambda: rng.random(m)}
+    cols = [gen_[f]() for f in fields]
+    eps = [rng.random(m) < 0.02 for _ in fields]
+    for c, e in zip(cols, eps):
+        c[e] = {"u1": 0xFF, "i4": -2**31, "i8": -2**63, "f4": np.nan, "f8": np.nan}[c.dtype.kind + str(c.itemsize)]
+    pos = rng.integers(-2, m + 3, n).astype(np.int32)
+    dts = [{"u8": vd.VD_U8, "i32": vd.VD_I32, "i64": vd.VD_I64, "f32": vd.VD_F32, "f64": vd.VD_F64}[f] for f in fields]
+    offs, stride = vd.row_layout(dts)
+    dcols = [cuda_tensor(c) for c in cols]
+    rows = torch.empty(m * stride, dtype=torch.uint8, device="cuda")
+    vd.zip_rows([vd.column(c) for c in dcols], rows)
+    outs = [torch.empty(max(n, 1), dtype=d.dtype, device="cuda") for d in dcols]
+    vd.gather_rows(rows, m, dts, cuda_tensor(pos), n, 1, outs)
+    assert vd.last_launch_count() == 1
+    # row bytes: each field at its offset, padding zero
+    rb = rows.cpu().numpy().reshape(m, stride)
+    for c, o in zip(cols, offs):
+        assert np.array_equal(rb[:, o:o + c.itemsize].copy().view(c.dtype).reshape(-1).view(np.uint8),
+                              c.view(np.uint8))
+    p_ = pos.astype(np.int64) - 1
+    p_[pos < 0] = -1
+    names = [f"f{k}" for k in range(len(fields))]
+    # Zip needs two or more inputs (Table 2); one field is a plain Gather
+    prog = (f"z := Zip({', '.join('t.' + x for x in names)})\ng := Gather(z, p)" if len(names) > 1
+            else "g := Gather(t.f0, p)")
+    po = oracle.run(prog, p=p_, **{f"t__{x}": (c.astype(np.float64 if c.dtype.kind == "f" else np.int64), e)
+                                    for x, c, e in zip(names, cols, eps)})
+    for x, c, o in zip(names, cols, outs):
+        vals, e = po.get_arrays(f"g.{x}" if len(names) > 1 else "g")
+        got = o[:n].cpu().numpy()
+        if c.dtype.kind == "f":
+            assert np.array_equal(np.isnan(got), e)
+            assert np.array_equal(got[~e].astype(np.float64), vals[~e])
+        else:
+            sentinel = {"uint8": 0xFF, "int32": -2**31, "int64": -2**63}[c.dtype.name]
+            assert np.array_equal(got.astype(np.int64), np.where(e, sentinel, vals).astype(np.int64))
+
+
 @pytest.mark.parametrize("n,out_len", [(0, 5), (1, 1), (5000, 100), (100000, 70000), (3, 0)])
 def test_scatter_last_writer_wins_vs_interpreter(n, out_len):
     rng = np.random.default_rng(n)
