@@ -45,7 +45,7 @@ def parse():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
     ap.add_argument("--workload", default="q1",
-                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14"])
+                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14", "q15"])
     ap.add_argument("--chunk", type=int, default=0,
                     help="select_unfused: rows per materialised chunk (0 = whole table; Fig 15 'Vectorized')")
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
@@ -67,7 +67,7 @@ def parse():
 
 
 def default_sf(w):
-    return {"q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0,
+    return {"q15": 100.0, "q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0,
             "select_unfused": 0.0, "fig14": 0.0}[w]
 
 
@@ -213,6 +213,8 @@ def main():
         return unfused_main(args, rank, world, local)
     if args.workload == "fig14":
         return fig14_main(args, rank, world, local)
+    if args.workload == "q15":
+        return q15_main(args, rank, world, local, sf)
 
     import torch
     import torch.distributed as dist
@@ -245,14 +247,7 @@ def main():
         return t
 
     def meta(t):
-        c = vd.column(t)
-        if c.dtype in (vd.VD_F32, vd.VD_F64) or t.numel() == 0:
-            return c
-        lo = torch.empty(1, dtype=t.dtype, device=dev)
-        hi = torch.empty(1, dtype=t.dtype, device=dev)
-        vd.fold_min(c, None, out=lo)
-        vd.fold_max(c, None, out=hi)
-        return vd.column(t, minmax=(int(lo.item()), int(hi.item())))
+        return vd.describe(t, stream=stream)
 
     dims, dim_views, cols = [], [], []
     if w == "q1":
@@ -676,6 +671,97 @@ def fig14_main(args, rank, world, local):
     if rank == 0:
         print(json.dumps(line), flush=True)
     comm.close()
+
+
+def q15_main(args, rank, world, local, sf):
+    """NEXT-4: TPC-H Q15's revenue view -- shipdate in [1996-01-01,
+    1996-04-01), GROUP BY l_suppkey (10,000 x SF groups: a key domain far
+    beyond a shared-memory table), SUM(ext * (100 - disc)), COUNT(*) --
+    through vd_group_fold (one streaming pass into the min/max-sized global
+    table + the FoldSelect compaction).  Algorithmic bytes: the four columns,
+    dense, 24 B/row (branching late loads touch fewer sectors)."""
+    import torch
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+
+    if world > 1:
+        if rank == 0:
+            print(json.dumps({"metric": METRIC, "workload": "q15", "unavailable": "q15 runs on one GPU "
+                              "(a cross-GPU merge of compacted high-cardinality groups is not implemented)"}))
+        return
+    torch.cuda.set_device(local % torch.cuda.device_count())
+    dev = torch.device("cuda", local % torch.cuda.device_count())
+    stream = torch.cuda.current_stream()
+    n = gen.lineitem_rows(sf)
+    names = ["l_shipdate", "l_suppkey", "l_extendedprice", "l_discount"]
+    cols = []
+    for nm in names:
+        col = gen.LINEITEM_COLS[nm]
+        t = torch.empty(n, dtype=getattr(torch, _dt(col)), device=dev)
+        gen.device(col, t.data_ptr(), n, 0, sf=sf, seed=args.seed, stream=stream.cuda_stream)
+        cols.append(t)
+    torch.cuda.synchronize()
+    views = [vd.describe(t, stream=stream) for t in cols]
+    p = vd.pred([[(0, ">=", 9496), (0, "<", 9587)]])
+    aggs = [("sum", [2, (3, 100, -1)]), ("count",)]
+    D = views[1].max - views[1].min + 1
+    keys = torch.empty(D, dtype=torch.int64, device=dev)
+    rows = torch.empty(D, dtype=torch.int64, device=dev)
+    slots = torch.empty(D * len(aggs) * 16, dtype=torch.uint8, device=dev)
+    ng = torch.empty(1, dtype=torch.int64, device=dev)
+    ws = vd.alloc_ws(vd.group_fold_ws_bytes(D, len(aggs)), dev)
+
+    def step():
+        vd.group_fold(views, n, 1, aggs, p, out_keys=keys, out_aggs=slots, out_rows=rows, out_ngroups=ng, ws=ws,
+                      stream=stream)
+
+    for _ in range(max(args.warmup, 3)):
+        step()
+    launches = vd.last_launch_count()
+    torch.cuda.synchronize()
+    steps = args.steps or 50
+    clocks = ClockSampler(local)
+    clocks.start()
+    time.sleep(0.3)
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    clk = clocks.stop()
+    ms = e0.elapsed_time(e1) / steps
+    g = int(ng.item())
+    digest = __import__("hashlib").sha256(keys[:g].cpu().numpy().tobytes() + rows[:g].cpu().numpy().tobytes() +
+                                          slots[:g * 32].cpu().numpy().tobytes()).hexdigest()[:16]
+    # algorithmic bytes of the branching plan: the filter column in full, and
+    # of every other column the 64-byte DRAM blocks holding a qualifying row
+    # (HBM's access granule; the dense figure, 24 B/row, is the predicated plan's)
+    mask = (cols[0] >= 9496) & (cols[0] < 9587)
+    alg_bytes = 4 * n
+    for t in cols[1:]:
+        r = 64 // t.element_size()
+        m = mask[:n // r * r].view(-1, r).any(1)
+        alg_bytes += 64 * (int(m.sum().item()) + int(bool(mask[n // r * r:].any().item())))
+    sel = float(mask.float().mean().item())
+    del mask
+    peak, kind = hbm_peak()
+    alg = alg_bytes / (ms * 1e-3) / 1e9
+    line = {"metric": METRIC, "value": n / (ms * 1e-3), "unit": "rows/s", "n_gpus": 1, "steps": steps,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "int64",
+            "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
+            "config": {"workload": f"tpch_q15_revenue_sf{sf:g}", "rows": n, "groups_domain": D, "groups": g,
+                       "sf": sf, "l2": f"inputs {n * 24 / 1e9:.1f} GB > 126 MB L2: no flush needed",
+                       "seed": args.seed},
+            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
+                         "peak_kind": kind, "traffic": ncu_traffic("q15"),
+                         "bytes_per_row": alg_bytes / n, "dense_bytes_per_row": 24, "selectivity": sel,
+                         "kernel": "vd_group_fold (k_grp_init + k_grp_fold + compaction)", "kernel_ms": ms},
+            "clocks": clk, "e2e": None, "gpu_launches": launches * steps, "result_digest": digest}
+    print(json.dumps(line), flush=True)
 
 
 def _dt(col):

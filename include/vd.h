@@ -72,8 +72,16 @@ typedef struct {
     int32_t scale;      /* decimal scale: value = data / 10^scale (0 = plain)  */
     int64_t min, max;   /* inclusive bounds of the non-epsilon values          */
     int32_t has_minmax; /* 1 if min/max are valid                              */
-    int32_t reserved;
+    int32_t flags;      /* VD_COL_* metadata bits (0 = nothing known)          */
 } vd_column;
+
+/* vd_column.flags: VD_COL_NOEPS -- the metadata producer has verified that
+ * no slot in [0, len) is epsilon (MonetDB's "nonil" column property).  Like
+ * min/max it is a promise by the caller; fused fragments use it (with
+ * min/max) to drop per-row epsilon / bounds checks.  A false promise gives
+ * unspecified results (never an out-of-bounds access: gathers still need
+ * min/max to prove their positions in range). */
+#define VD_COL_NOEPS 1
 
 /* Control vector (§2.2 Controlled Folding).  Runs = maximal
  * blocks of ADJACENT equal values (reading A3).
@@ -176,7 +184,8 @@ vd_status vd_workspace_bytes(int32_t op, int64_t n, const vd_ctrl* ctrl, const s
  * `dev_dst` (async on `stream`; `host_src` should be pinned for overlap) and
  * fill the view *out (data = dev_dst).  If compute_minmax != 0 the value
  * bounds are computed on the host from host_src while the copy runs and
- * stored in out->min/max (epsilon values excluded; floats: has_minmax = 0). */
+ * stored in out->min/max (epsilon values excluded; floats: has_minmax = 0),
+ * and VD_COL_NOEPS is set in out->flags if no slot is epsilon. */
 vd_status vd_load_column(const void* host_src, int64_t len, int32_t dtype, int32_t scale, void* dev_dst,
                          int32_t compute_minmax, void* stream, vd_column* out);
 
@@ -372,6 +381,37 @@ size_t vd_partials_bytes(const vd_pipeline* plan);
 vd_status vd_run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_t ncols, int64_t n,
                           const vd_column* dims, int32_t ndims, void* out_partials, void* ws, size_t ws_bytes,
                           void* stream);
+
+/* Grouped fold over a LARGE key domain.  The
+ * paper's frontend sizes grouping tables from min/max metadata and
+ * addresses them by identity hashing: row i belongs to group
+ * key[i] - key.min in [0, D), D = key.max - key.min + 1 (<= VD_MAX_DOMAIN).
+ * Fig 10/11's chain Partition -> Scatter -> FoldSum/FoldCount/... ->
+ * FoldSelect compaction with the Partition/Scatter virtual
+ * (§3.1.3): every qualifying row folds into a D-slot table in the
+ * workspace (global reductions: the shared-memory tables of
+ * vd_run_pipeline spilled), then the non-empty slots are compacted.
+ *   cols[0..ncols), n, pred : as vd_run_pipeline (no gathers); epsilon
+ *       never qualifies (A9).
+ *   key_col : an i32/i64 column WITH min/max metadata (VD_E_DOMAIN
+ *       without); an epsilon key has no group.
+ *   aggs[0..naggs) : SUM (integer: exact, int64 table slots proven from
+ *       the factors' min/max x n, else VD_E_OVERFLOW; float: f64, summed
+ *       in an unspecified order), COUNT(*), MIN / MAX (integer only).  An
+ *       epsilon factor makes the row's value epsilon: skipped (A5).
+ *   outputs (device, capacity D groups; only *out_ngroups are written), in
+ *       ascending key order with empty groups dropped (A16):
+ *       out_keys[g] int64, out_aggs[g*naggs + a] 16-byte slots as in
+ *       vd_partials (integer SUM/COUNT: int128; MIN/MAX: int64 sign-
+ *       extended, epsilon INT64_MIN if the group had no non-epsilon value;
+ *       float SUM: f64 in the low 8 bytes), out_rows[g] int64 row count,
+ *       *out_ngroups_dev int64.
+ *   ws : vd_group_fold_ws_bytes(D, naggs) bytes. */
+#define VD_MAX_DOMAIN ((int64_t)1 << 31)
+vd_status vd_group_fold_ws_bytes(int64_t domain, int32_t naggs, size_t* bytes_host);
+vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const vd_pred* pred, int32_t key_col,
+                        const vd_agg* aggs, int32_t naggs, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
+                        int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
 
 /* Host merge of per-device partials (rank order, exact 128-bit / f64), the
  * cross-GPU step of the hierarchical fold (Fig 3 one level up):

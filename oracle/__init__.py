@@ -9,7 +9,7 @@ Layer 1 -- :class:`Program`: a literal interpreter of Voodoo programs
 (§2.2 Table 2) over epsilon-padded vectors, every
 intermediate materialised (the paper's interpreter).
 
-Layer 2 -- :func:`q1`, :func:`q6`, :func:`select_f32`, :func:`fkj`:
+Layer 2 -- :func:`q1`, :func:`q6`, :func:`q15`, :func:`select_f32`, :func:`fkj`:
 brute-force SQL-equivalent loops (TPC-H SQL [ext]) written independently of
 layer 1.  Both layers are plain single-threaded C++17 (``liboracle.so``).
 
@@ -53,6 +53,8 @@ def _lib():
         L.or_ctx_get_f64.argtypes = [vp, c, vp, vp, vp]
         L.or_q1.argtypes = [i64, vp, vp, vp, vp, vp, vp, vp, ctypes.c_int32, vp, vp]
         L.or_q6.argtypes = [i64, vp, vp, vp, vp, ctypes.c_int32, ctypes.c_int32, i64, i64, i64, vp, vp, vp]
+        L.or_q15.argtypes = [i64, vp, vp, vp, vp, ctypes.c_int32, ctypes.c_int32, vp, vp, vp, vp]
+        L.or_q15.restype = i64
         L.or_select_f32.argtypes = [i64, vp, ctypes.c_float, ctypes.c_int, vp, vp, vp]
         L.or_select_f32.restype = i64
         L.or_fkj.argtypes = [ctypes.c_int, i64] + [vp] * 8 + [i64, vp, vp, vp, i64, vp, vp, vp]
@@ -197,6 +199,20 @@ def q6(cols: Dict[str, np.ndarray], d0: int = 8766, d1: int = 9131, dlo: int = 5
     _lib().or_q6(n, _p(a["l_shipdate"]), _p(a["l_discount"]), _p(a["l_quantity"]), _p(a["l_extendedprice"]),
                  int(d0), int(d1), int(dlo), int(dhi), int(qmax), _p(lo), _p(hi), _p(cnt))
     return _to_int(lo[0], hi[0]), int(cnt[0])
+
+
+def q15(cols: Dict[str, np.ndarray], d0: int = 9496, d1: int = 9587):
+    """Brute-force TPC-H Q15 revenue view: {suppkey: (revenue exact int scale 1e4, count)}
+    for ship in [d0, d1) (default [1996-01-01, 1996-04-01))."""
+    n = len(cols["l_shipdate"])
+    key = np.zeros(max(n, 1), dtype=np.int64)
+    lo = np.zeros(max(n, 1), dtype=np.int64)
+    hi = np.zeros(max(n, 1), dtype=np.int64)
+    cnt = np.zeros(max(n, 1), dtype=np.int64)
+    a = {k: np.ascontiguousarray(cols[k]) for k in ("l_shipdate", "l_suppkey", "l_extendedprice", "l_discount")}
+    g = _lib().or_q15(n, _p(a["l_shipdate"]), _p(a["l_suppkey"]), _p(a["l_extendedprice"]), _p(a["l_discount"]),
+                      int(d0), int(d1), _p(key), _p(lo), _p(hi), _p(cnt))
+    return {int(key[j]): (_to_int(lo[j], hi[j]), int(cnt[j])) for j in range(g)}
 
 
 def select_f32(v: np.ndarray, t: float, op: str = "lt", want_positions: bool = True):

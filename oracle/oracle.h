@@ -57,6 +57,12 @@ void or_q1(int64_t n, const int32_t* ship, const uint8_t* rf, const uint8_t* ls,
  * qty < qmax. out[0] = revenue (scale 1e4, 128-bit lo/hi), *count. */
 void or_q6(int64_t n, const int32_t* ship, const int64_t* disc, const int64_t* qty, const int64_t* ext, int32_t d0,
            int32_t d1, int64_t dlo, int64_t dhi, int64_t qmax, int64_t* rev_lo, int64_t* rev_hi, int64_t* count);
+/* TPC-H Q15 revenue view: for rows with ship in [d0, d1), group by suppkey
+ * (ascending, only keys that occur): out_key[g], revenue sum(ext*(100-disc))
+ * (scale 1e4, 128-bit lo/hi), out_cnt[g] rows.  Capacity n groups; returns
+ * the number of groups. */
+int64_t or_q15(int64_t n, const int32_t* ship, const int32_t* suppkey, const int64_t* ext, const int64_t* disc,
+               int32_t d0, int32_t d1, int64_t* out_key, int64_t* out_lo, int64_t* out_hi, int64_t* out_cnt);
 /* Float selection micro-benchmark (Fig 1): positions i (ascending)
  * with v[i] < t (op=0) or v[i] > t (op=1); returns count, writes positions
  * and the long-double sum of selected values (split into hi + lo doubles). */

@@ -62,6 +62,41 @@ extern "C" void or_q6(int64_t n, const int32_t* ship, const int64_t* disc, const
     *count = c;
 }
 
+extern "C" int64_t or_q15(int64_t n, const int32_t* ship, const int32_t* suppkey, const int64_t* ext,
+                          const int64_t* disc, int32_t d0, int32_t d1, int64_t* out_key, int64_t* out_lo,
+                          int64_t* out_hi, int64_t* out_cnt) {
+    // TPC-H Q15's revenue view [ext]: shipdate in [DATE, DATE + 3 months),
+    // GROUP BY l_suppkey, SUM(l_extendedprice * (1 - l_discount)) -- here
+    // ext * (100 - disc) at scale 1e4 (reading A17).  A std::map keyed by the
+    // supplier key: ascending key order, only suppliers that occur (the
+    // SQL GROUP BY result, reading A16).  Returns the number of groups.
+    // collect the qualifying (key, value) pairs, stable-sort by key, sum runs
+    std::vector<std::pair<int64_t, i128>> rows;
+    for (int64_t i = 0; i < n; ++i)
+        if (ship[i] >= d0 && ship[i] < d1) rows.push_back({(int64_t)suppkey[i], (i128)ext[i] * (100 - disc[i])});
+    std::stable_sort(rows.begin(), rows.end(),
+                     [](const std::pair<int64_t, i128>& a, const std::pair<int64_t, i128>& b) { return a.first < b.first; });
+    int64_t g = -1;
+    i128 rev = 0;
+    int64_t cnt = 0;
+    for (size_t k = 0; k <= rows.size(); ++k) {
+        if (k == rows.size() || (k > 0 && rows[k].first != rows[k - 1].first)) {
+            if (k > 0) {
+                ++g;
+                out_key[g] = rows[k - 1].first;
+                put128(rev, &out_lo[g], &out_hi[g]);
+                out_cnt[g] = cnt;
+            }
+            rev = 0;
+            cnt = 0;
+        }
+        if (k == rows.size()) break;
+        rev += rows[k].second;
+        ++cnt;
+    }
+    return g + 1;
+}
+
 extern "C" int64_t or_select_f32(int64_t n, const float* v, float t, int op, int32_t* pos, double* sum_hi,
                                  double* sum_lo) {
     // Fig 1: filter a list of values with a predicate; the output

@@ -1440,6 +1440,7 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
             } else {
                 v = x * (a.a + a.b * y);
             }
+            if (x == INT64_MIN || y == INT64_MIN) v = 0;  // epsilon factor: skipped by SUM (A5/A9)
         }
         return key;
     };
@@ -1591,6 +1592,239 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
     if (!s_last) return;
     __threadfence();
     for (int k = threadIdx.x; k < NS; k += FKG_THREADS) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
+            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[k], t);
+    }
+}
+
+// ---- FK grouped fold with per-thread private group slots ----------------------
+// The same Q9-shaped fragment when the host proves from min/max metadata that
+// every row's value X*(a+bY) lies in [0, 2^31) and the key part B is a
+// calendar year inside 1969..2099: each consumer thread owns one packed u64
+// slot per group in shared memory, laid out [group][thread] (a warp's 32
+// lanes always touch 32 consecutive u64 words: conflict-free whatever the
+// keys), holding sum + (count << 48).  A row is one LDS.64 / IADD.64 / STS.64
+// -- no atomics, no leader election -- and the group table of the virtual
+// scatter (§3.1.3) is private down to the work item, the Fig 3
+// hierarchy with one more level.  The host bounds the rows per thread to
+// < 2^16 (grid size), so the 16-bit count and 48-bit sum cannot carry.
+// CHECKED = false when metadata also proves that every row joins (FK inside
+// the dimension, no epsilon) and every key lies in [0, ngroups): then no row
+// needs the trash slot and the checks compile away.
+// The year comes from (4(d+365)+3) / 1461 + 1969 (exact for 1969-01-01 ..
+// 2099-12-31; the host checks the column's range).
+constexpr int FKP_TILE = 1024;
+constexpr int FKP_CW = 4;
+constexpr int FKP_NT = FKP_CW * 32;
+constexpr int FKP_THREADS = FKP_NT + 32;
+constexpr int FKP_RPT = FKP_TILE / FKP_NT;  // 8 rows per thread per tile, as 4 row pairs
+constexpr int FKP_MAXSLOTS = 176;           // ngroups (+ trash) that fit beside a 2-stage ring
+constexpr int FKP_STAGES = 2;
+
+template <bool CHECKED, int BATCH>
+__global__ void __launch_bounds__(FKP_THREADS, 1) k_pipe_fkg_priv(const __grid_constant__ FkgArgs a, int64_t ntiles,
+                                                                  int32_t pf_dist, Slot16* __restrict__ parts,
+                                                                  unsigned int* __restrict__ done,
+                                                                  Slot16* __restrict__ out) {
+    extern __shared__ __align__(128) uint8_t smem[];
+    constexpr int SB = FKP_TILE * (4 + 4 + 8 + 8);
+    const int GS = a.ngroups + (CHECKED ? 1 : 0);
+    uint64_t* tab = reinterpret_cast<uint64_t*>(smem + (size_t)FKP_STAGES * SB);  // [GS][FKP_NT]
+    uint64_t* full = tab + (size_t)GS * FKP_NT;
+    uint64_t* empty = full + FKP_STAGES;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int s = 0; s < FKP_STAGES; ++s) {
+            mbar_init(&full[s], 1);
+            mbar_init(&empty[s], FKP_CW);
+        }
+        fence_mbar_init();
+    }
+    for (int k = threadIdx.x; k < GS * FKP_NT; k += FKP_THREADS) tab[k] = 0;
+    __syncthreads();
+
+    constexpr uint64_t ONE = 1ull << 48;
+    // key of a row from its dimension value d and base key column value kb
+    auto keyof = [&](int d, int32_t kb) -> int {
+        const int kbv = a.yfn ? (4 * (kb + 365) + 3) / 1461 + 1969 : kb;
+        int key = (d - a.subA) * a.mA + (kbv - a.subB) * a.mB;
+        if (CHECKED) {
+            if (d == 0x100 || d == 0xFF || kb == INT32_MIN || key < 0 || key >= a.ngroups) key = a.ngroups;
+        }
+        return key;
+    };
+    auto gather = [&](int32_t fk) -> int {
+        const int64_t p = (int64_t)fk - a.bias;
+        if (CHECKED) return (fk != INT32_MIN && p >= 0 && p < a.dim_len) ? (int)__ldg(a.dim + p) : 0x100;
+        return (int)__ldg(a.dim + p);
+    };
+    // an epsilon factor makes the row's value epsilon: skipped by the SUM
+    // (reading A5/A9), still counted by COUNT(*)
+    auto value = [&](int64_t x, int64_t y) -> uint64_t {
+        const int32_t f = (int32_t)((uint32_t)a.a + (uint32_t)a.b * (uint32_t)y);
+        const uint64_t v = (uint64_t)((uint32_t)x) * (uint64_t)(uint32_t)f;  // both proven in [0, 2^31)
+        if (CHECKED) return (x == INT64_MIN || y == INT64_MIN) ? 0ull : v;
+        return v;
+    };
+    uint64_t* mytab = tab + threadIdx.x;
+    auto fold = [&](int key, uint64_t v) {
+        uint64_t* p = mytab + (size_t)key * FKP_NT;
+        *p += v + ONE;
+    };
+
+    if (warp == FKP_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = blockIdx.x + it * gridDim.x;
+                if (tile >= ntiles) break;
+                const int s = (int)(it % FKP_STAGES);
+                if (pf_dist > 0) {
+                    const int64_t pt = tile + (int64_t)pf_dist * gridDim.x;
+                    if (pt < ntiles) {
+                        const int64_t q0 = pt * FKP_TILE;
+                        prefetch_l2_bulk(a.fk + q0, FKP_TILE * 4);
+                        prefetch_l2_bulk(a.kb + q0, FKP_TILE * 4);
+                        prefetch_l2_bulk(a.x + q0, FKP_TILE * 8);
+                        prefetch_l2_bulk(a.y + q0, FKP_TILE * 8);
+                    }
+                }
+                if (it >= FKP_STAGES) mbar_wait(&empty[s], (uint32_t)(((it / FKP_STAGES) - 1) & 1));
+                uint8_t* st = smem + (size_t)s * SB;
+                const int64_t r0 = tile * FKP_TILE;
+                mbar_expect_tx(&full[s], SB);
+                tma_load_1d(st, a.fk + r0, FKP_TILE * 4, &full[s], pol);
+                tma_load_1d(st + FKP_TILE * 4, a.kb + r0, FKP_TILE * 4, &full[s], pol);
+                tma_load_1d(st + FKP_TILE * 8, a.x + r0, FKP_TILE * 8, &full[s], pol);
+                tma_load_1d(st + FKP_TILE * 16, a.y + r0, FKP_TILE * 8, &full[s], pol);
+            }
+        }
+        __syncwarp();
+    } else {
+        // software pipeline: the gathers of tile i are issued before tile i-1
+        // (whose gathers flew during the previous iteration) is folded
+        // two tiles of gathers in flight: a tile's gathers are issued, then the
+        // tile two iterations back is folded (its gathers have had two
+        // iterations to return); pd/pkb/pv hold that oldest tile, qd/qkb/qv
+        // the one in between
+        int pd[FKP_RPT], pkb[FKP_RPT], qd[FKP_RPT], qkb[FKP_RPT];
+        uint64_t pv[FKP_RPT], qv[FKP_RPT];
+        int have = 0;
+        // the RPT read-modify-writes of a batch are independent unless two rows
+        // share a key: all loads issue first, a row whose key repeats an
+        // earlier row's takes that row's updated value (register selects, no
+        // shared-memory round trip), and the stores go out in row order so
+        // the last one to an address carries the full sum
+        auto drain = [&]() {
+#pragma unroll
+            for (int b0 = 0; b0 < FKP_RPT; b0 += BATCH) {
+                int key[BATCH];
+                uint64_t t[BATCH];
+#pragma unroll
+                for (int k = 0; k < BATCH; ++k) {
+                    key[k] = keyof(pd[b0 + k], pkb[b0 + k]);
+                    t[k] = mytab[(size_t)key[k] * FKP_NT];
+                }
+#pragma unroll
+                for (int k = 0; k < BATCH; ++k) {
+                    uint64_t b = t[k];
+#pragma unroll
+                    for (int j = 0; j < k; ++j) b = (key[j] == key[k]) ? t[j] : b;
+                    t[k] = b + pv[b0 + k] + ONE;
+                }
+#pragma unroll
+                for (int k = 0; k < BATCH; ++k) mytab[(size_t)key[k] * FKP_NT] = t[k];
+            }
+        };
+        for (int64_t it = 0;; ++it) {
+            const int64_t tile = blockIdx.x + it * gridDim.x;
+            if (tile >= ntiles) break;
+            const int s = (int)(it % FKP_STAGES);
+            mbar_wait(&full[s], (uint32_t)((it / FKP_STAGES) & 1));
+            const uint8_t* st = smem + (size_t)s * SB;
+            int32_t f[FKP_RPT], kb[FKP_RPT];
+            uint64_t v[FKP_RPT];
+#pragma unroll
+            for (int k = 0; k < FKP_RPT / 2; ++k) {
+                const int r = 2 * threadIdx.x + k * 2 * FKP_NT;  // a row pair
+                const int2 fk2 = *reinterpret_cast<const int2*>(st + (size_t)r * 4);
+                const int2 kb2 = *reinterpret_cast<const int2*>(st + FKP_TILE * 4 + (size_t)r * 4);
+                const longlong2 x2 = *reinterpret_cast<const longlong2*>(st + FKP_TILE * 8 + (size_t)r * 8);
+                const longlong2 y2 = *reinterpret_cast<const longlong2*>(st + FKP_TILE * 16 + (size_t)r * 8);
+                f[2 * k] = fk2.x; f[2 * k + 1] = fk2.y;
+                kb[2 * k] = kb2.x; kb[2 * k + 1] = kb2.y;
+                v[2 * k] = value(x2.x, y2.x);
+                v[2 * k + 1] = value(x2.y, y2.y);
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[s]);
+            int d[FKP_RPT];
+#pragma unroll
+            for (int k = 0; k < FKP_RPT; ++k) d[k] = gather(f[k]);
+            if (have == 2) drain();
+#pragma unroll
+            for (int k = 0; k < FKP_RPT; ++k) {
+                pd[k] = qd[k]; pkb[k] = qkb[k]; pv[k] = qv[k];
+                qd[k] = d[k]; qkb[k] = kb[k]; qv[k] = v[k];
+            }
+            have = have < 2 ? have + 1 : 2;
+        }
+        if (have == 2) drain();
+        if (have >= 1) {
+#pragma unroll
+            for (int k = 0; k < FKP_RPT; ++k) { pd[k] = qd[k]; pkb[k] = qkb[k]; pv[k] = qv[k]; }
+            drain();
+        }
+        if (blockIdx.x == 0) {
+            // ragged tail (< one tile): direct loads, always checked
+            for (int64_t r = ntiles * FKP_TILE + threadIdx.x; r < a.n; r += FKP_NT) {
+                const int32_t fk = a.fk[r], kbr = a.kb[r];
+                const int64_t p = (int64_t)fk - a.bias;
+                const int d = (fk != INT32_MIN && p >= 0 && p < a.dim_len) ? (int)a.dim[p] : 0x100;
+                const int kbv = a.yfn ? (4 * (kbr + 365) + 3) / 1461 + 1969 : kbr;
+                const int key = (d - a.subA) * a.mA + (kbv - a.subB) * a.mB;
+                const bool ok = !(d == 0x100 || d == 0xFF || kbr == INT32_MIN || key < 0 || key >= a.ngroups);
+                if (ok) {
+                    const int64_t xr = a.x[r], yr = a.y[r];
+                    const int32_t f = (int32_t)((uint32_t)a.a + (uint32_t)a.b * (uint32_t)yr);
+                    const uint64_t v = (xr == INT64_MIN || yr == INT64_MIN)
+                                           ? 0ull : (uint64_t)((uint32_t)xr) * (uint64_t)(uint32_t)f;
+                    fold(key, v);
+                }
+            }
+        }
+    }
+    __syncthreads();
+    // CTA fold: per group, the 128 private slots -> (sum, count), int128 into
+    // [ngroups][naggs+1] in the plan's layout
+    const int NS = a.ngroups * (a.naggs + 1);
+    for (int k = threadIdx.x; k < NS; k += FKP_THREADS) {
+        const int g = k / (a.naggs + 1), ag = k % (a.naggs + 1);
+        const bool cnt = (ag == a.naggs || ag == a.cnt_slot);
+        const uint64_t* row = tab + (size_t)g * FKP_NT;
+        uint64_t t = 0;
+        for (int j = 0; j < FKP_NT; ++j) {
+            const uint64_t w = row[(j + threadIdx.x) & (FKP_NT - 1)];  // rotated start: spread banks
+            t += cnt ? (w >> 48) : (w & (ONE - 1));
+        }
+        put_i128(&parts[(size_t)blockIdx.x * NS + k], (i128)t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    for (int k = threadIdx.x; k < NS; k += FKP_THREADS) {
         i128 t = 0;
         for (unsigned b = 0; b < gridDim.x; ++b) {
             Slot16 x;
@@ -2661,6 +2895,66 @@ static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols,
     }
     A.ngroups = (int32_t)p->ngroups;
     A.n = n;
+    // ---- private-slot variant (k_pipe_fkg_priv): values proven in [0, 2^31)
+    {
+        const double flo = std::min((double)A.a + (double)A.b * by.lo, (double)A.a + (double)A.b * by.hi);
+        const vd_column &cfk = cols[fkcol], &ckb = cols[kbcol];
+        const bool yr_ok = !A.yfn || (ckb.has_minmax && ckb.min >= -365 && ckb.max <= 47481);
+        const bool fits = narrow && bx.lo >= 0 && flo >= 0 && xmx * fmx < 2147483647.0 && yr_ok;
+        auto noeps = [](const vd_column& c) { return (c.flags & VD_COL_NOEPS) != 0; };
+        bool proven = fits && noeps(cfk) && noeps(ckb) && noeps(cols[X]) && noeps(cols[Y]) && noeps(dim) &&
+                      cfk.has_minmax && dim.has_minmax && ckb.has_minmax && cfk.min - gs.bias >= 0 &&
+                      cfk.max - gs.bias < dim.len && dim.max < 0xFF;
+        if (proven) {
+            // key range over the corners of (d, kb') from metadata
+            const int64_t k0 = A.yfn ? (4 * (ckb.min + 365) + 3) / 1461 + 1969 : ckb.min;
+            const int64_t k1 = A.yfn ? (4 * (ckb.max + 365) + 3) / 1461 + 1969 : ckb.max;
+            int64_t kmin = INT64_MAX, kmax = INT64_MIN;
+            for (int64_t d : {dim.min, dim.max})
+                for (int64_t kk : {k0, k1}) {
+                    const int64_t key = (d - A.subA) * (int64_t)A.mA + (kk - A.subB) * (int64_t)A.mB;
+                    kmin = std::min(kmin, key);
+                    kmax = std::max(kmax, key);
+                }
+            proven = kmin >= 0 && kmax < A.ngroups;
+        }
+        const int slots = A.ngroups + (proven ? 0 : 1);
+        const int64_t ntiles = n / FKP_TILE;
+        // rows per private slot set < 2^16: tiles per CTA * 8 + tail 8
+        const int64_t grid = std::max<int64_t>(num_sms(), (ntiles + 8000 - 1) / 8000);
+        // opt-in (VD_FKG_VARIANT=priv): one consumer warp per scheduler leaves
+        // its dependency chains exposed -- 4.6 ms vs 3.3 ms for the
+        // shared-atomic kernel at Q9 SF100 (profiles/round1_q9.md)
+        const bool want_priv = var && strcmp(var, "priv") == 0;
+        if (want_priv && fits && slots <= FKP_MAXSLOTS && grid <= grid_persistent(4)) {
+            const size_t smem = (size_t)FKP_STAGES * FKP_TILE * 24 + (size_t)slots * FKP_NT * 8 + 2 * FKP_STAGES * 8;
+            const char* pfv = getenv("VD_FKP_PF");
+            const int32_t pf = pfv ? atoi(pfv) : 0;
+            unsigned int* dn = (unsigned int*)ws;
+            Slot16* parts = (Slot16*)((char*)ws + 256);
+            cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+            if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+            auto go = [&](auto kern) {
+                cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+                kern<<<(unsigned)grid, FKP_THREADS, smem, s>>>(A, ntiles, pf, parts, dn, (Slot16*)out);
+            };
+            const char* bv = getenv("VD_FKP_BATCH");
+            const int batch = bv ? atoi(bv) : 4;
+            if (proven) {
+                if (batch == 8) go(k_pipe_fkg_priv<false, 8>);
+                else if (batch == 2) go(k_pipe_fkg_priv<false, 2>);
+                else go(k_pipe_fkg_priv<false, 4>);
+            } else {
+                go(k_pipe_fkg_priv<true, 4>);
+            }
+            ++*nl;
+            e = cudaGetLastError();
+            if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+            set_fragment(proven ? "fk_group_priv" : "fk_group_priv_checked");
+            *done = true;
+            return VD_OK;
+        }
+    }
     constexpr size_t SB = FKG_TILE * 24;
     const size_t fixed = (size_t)FKG_CW * 3 * (((size_t)p->ngroups + 32) & ~(size_t)31) * 4 + FKG_CW * 32 * 8 + (size_t)((A.ydays + 7) & ~7) * 2 +
                          2 * GF_MAXSTAGES * 8;

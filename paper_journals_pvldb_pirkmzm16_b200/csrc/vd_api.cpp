@@ -352,16 +352,18 @@ vd_status vd_load_column(const void* host_src, int64_t len, int32_t dtype, int32
         // such min/max metadata per column)
         int64_t mn = INT64_MAX, mx = INT64_MIN;
         bool any = false;
+        int64_t neps = 0;
         for (int64_t i = 0; i < len; ++i) {
             int64_t v;
-            if (dtype == VD_U8) { uint8_t x = ((const uint8_t*)host_src)[i]; if (x == VD_EPS_U8) continue; v = x; }
-            else if (dtype == VD_I32) { int32_t x = ((const int32_t*)host_src)[i]; if (x == VD_EPS_I32) continue; v = x; }
-            else { int64_t x = ((const int64_t*)host_src)[i]; if (x == VD_EPS_I64) continue; v = x; }
+            if (dtype == VD_U8) { uint8_t x = ((const uint8_t*)host_src)[i]; if (x == VD_EPS_U8) { ++neps; continue; } v = x; }
+            else if (dtype == VD_I32) { int32_t x = ((const int32_t*)host_src)[i]; if (x == VD_EPS_I32) { ++neps; continue; } v = x; }
+            else { int64_t x = ((const int64_t*)host_src)[i]; if (x == VD_EPS_I64) { ++neps; continue; } v = x; }
             mn = std::min(mn, v);
             mx = std::max(mx, v);
             any = true;
         }
         if (any) { out->min = mn; out->max = mx; out->has_minmax = 1; }
+        if (neps == 0) out->flags |= VD_COL_NOEPS;
     }
     return VD_OK;
 }
@@ -625,6 +627,79 @@ vd_status vd_run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_
     if ((st = check_device()) != VD_OK) return st;
     int nl = 0;
     st = run_pipeline(plan, cols, ncols, n, dims, ndims, out, ws, ws_bytes, (cudaStream_t)stream, &nl);
+    count_launches(nl);
+    return st;
+}
+
+// ---- NEXT-4: grouped fold over a large key domain (k_group.cu) --------------
+vd_status vd_group_fold_ws_bytes(int64_t domain, int32_t naggs, size_t* bytes) {
+    if (!bytes) return VD_E_NULL;
+    if (domain < 1 || domain > VD_MAX_DOMAIN || naggs < 0 || naggs > VD_MAX_AGGS) return VD_E_ARG;
+    *bytes = group_ws_bytes(domain, naggs);
+    return VD_OK;
+}
+
+vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const vd_pred* pred, int32_t key_col,
+                        const vd_agg* aggs, int32_t naggs, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
+                        int64_t* out_ngroups, void* ws, size_t ws_bytes, void* stream) {
+    reset_launches();
+    if (n < 0) return VD_E_SHAPE;
+    if (ncols < 1 || ncols > VD_MAX_DEVCOLS || !cols) { set_error("group_fold: columns"); return VD_E_ARG; }
+    if (naggs < 0 || naggs > VD_MAX_AGGS || (naggs > 0 && !aggs)) { set_error("group_fold: naggs in [0, 8]"); return VD_E_ARG; }
+    if (!out_keys || !out_rows || !out_ngroups || (naggs > 0 && !out_aggs)) { set_error("group_fold: outputs"); return VD_E_NULL; }
+    vd_status st;
+    DevCols dc;
+    std::memset(&dc, 0, sizeof(dc));
+    dc.ncols = ncols;
+    for (int c = 0; c < ncols; ++c) {
+        if ((st = check_col(&cols[c], n, "group_fold")) != VD_OK) return st;
+        dc.p[c] = cols[c].data;
+        dc.dt[c] = cols[c].dtype;
+    }
+    if ((st = check_pred(pred, dc.dt, ncols)) != VD_OK) return st;
+    if (key_col < 0 || key_col >= ncols) { set_error("group_fold: key column out of range"); return VD_E_ARG; }
+    const vd_column& kc = cols[key_col];
+    if (kc.dtype != VD_I32 && kc.dtype != VD_I64) { set_error("group_fold: key must be i32/i64"); return VD_E_DTYPE; }
+    // identity hashing: the table is sized from the key's min/max
+    if (!kc.has_minmax) { set_error("group_fold: the key column needs min/max metadata"); return VD_E_DOMAIN; }
+    const double dspan = (double)kc.max - (double)kc.min + 1.0;
+    if (kc.max < kc.min || dspan > (double)VD_MAX_DOMAIN) { set_error("group_fold: key domain exceeds VD_MAX_DOMAIN"); return VD_E_DOMAIN; }
+    const int64_t D = kc.max - kc.min + 1;
+    int32_t isf[VD_MAX_AGGS] = {0};
+    for (int a = 0; a < naggs; ++a) {
+        const vd_agg& g = aggs[a];
+        if (g.kind < VD_AGG_SUM || g.kind > VD_AGG_MAX) { set_error("bad aggregate kind"); return VD_E_ARG; }
+        if (g.kind == VD_AGG_COUNT) continue;
+        if (g.nfactors < 1 || g.nfactors > VD_MAX_FACTORS) { set_error("nfactors in [1, 3]"); return VD_E_ARG; }
+        double mx = 1.0;  // bound of |product|
+        bool known = true;
+        for (int f = 0; f < g.nfactors; ++f) {
+            const vd_factor& fc = g.f[f];
+            if (fc.col < -1 || fc.col >= ncols) { set_error("factor column out of range"); return VD_E_ARG; }
+            if (fc.col < 0) { mx *= std::fabs((double)fc.a); continue; }
+            const vd_column& c = cols[fc.col];
+            if (c.dtype == VD_F32 || c.dtype == VD_F64) { isf[a] = 1; continue; }
+            if (!c.has_minmax) { known = false; continue; }
+            const double x1 = (double)fc.a + (double)fc.b * (double)c.min, x2 = (double)fc.a + (double)fc.b * (double)c.max;
+            mx *= std::max(std::fabs(x1), std::fabs(x2));
+        }
+        if (isf[a] && g.kind != VD_AGG_SUM) { set_error("group_fold: float MIN/MAX not supported"); return VD_E_UNSUPPORTED; }
+        if (isf[a]) continue;
+        // int64 table slots: a SUM must be exact over all n rows, MIN/MAX must
+        // stay below the table's identity values
+        const double lim = g.kind == VD_AGG_SUM ? mx * (double)(n > 0 ? n : 1) : mx;
+        if (!known || lim >= 9.2e18) {
+            set_error("group_fold: min/max metadata cannot prove int64 aggregates exact");
+            return VD_E_OVERFLOW;
+        }
+    }
+    if ((st = check_ws(ws, ws_bytes, group_ws_bytes(D, naggs))) != VD_OK) return st;
+    if ((st = check_device()) != VD_OK) return st;
+    DevPred dp;
+    make_devpred(pred, &dp);
+    int nl = 0;
+    st = cuda_status(launch_group_fold(dc, dp, n, key_col, kc.min, D, aggs, isf, naggs, out_keys, out_aggs, out_rows,
+                                       out_ngroups, ws, (cudaStream_t)stream, &nl));
     count_launches(nl);
     return st;
 }

@@ -212,4 +212,10 @@ __device__ __forceinline__ void tma_load_1d(void* smem_dst, const void* gsrc, ui
         : "memory");
 }
 
+// Bulk prefetch global -> L2 (no shared-memory destination, no completion):
+// keeps HBM requests in flight beyond what the shared-memory ring can hold.
+__device__ __forceinline__ void prefetch_l2_bulk(const void* gsrc, uint32_t bytes) {
+    asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(gsrc), "r"(bytes) : "memory");
+}
+
 }  // namespace vd

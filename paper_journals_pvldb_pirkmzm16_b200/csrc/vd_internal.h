@@ -97,6 +97,13 @@ vd_status run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_t n
                        const vd_column* dims, int32_t ndims, void* out, void* ws, size_t ws_bytes, cudaStream_t s,
                        int* nlaunch);
 
+// k_group.cu (NEXT-4)
+size_t group_ws_bytes(int64_t D, int naggs);
+cudaError_t launch_group_fold(const DevCols& cols, const DevPred& pred, int64_t n, int key_col, int64_t kmin,
+                              int64_t D, const vd_agg* aggs, const int32_t* isf, int naggs, int64_t* out_keys,
+                              void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws, cudaStream_t s,
+                              int* nl);
+
 int num_sms();
 
 }  // namespace vd

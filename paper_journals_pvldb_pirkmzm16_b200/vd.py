@@ -34,6 +34,7 @@ VD_SEL_BRANCH, VD_SEL_PREDICATED, VD_SEL_PREDICATED_LOOKUP = 0, 1, 2
 VD_OP_SELECT, VD_OP_FOLD, VD_OP_SCATTER, VD_OP_PIPELINE, VD_OP_FOLD_SELECT, VD_OP_PARTITION = range(6)
 VD_AGG_SUM, VD_AGG_COUNT, VD_AGG_MIN, VD_AGG_MAX = range(4)
 VD_SCATTER_UNIQUE = 1
+VD_COL_NOEPS = 1
 VD_MAX_TERMS, VD_MAX_CONJ, VD_MAX_AGGS, VD_MAX_FACTORS, VD_MAX_GATHERS, VD_MAX_KEYPARTS = 8, 4, 8, 3, 4, 3
 VD_WS_DOMAIN_ERRORS_OFFSET = 128
 
@@ -47,7 +48,7 @@ CMP = {">": VD_CMP_GT, "<": VD_CMP_LT, "==": VD_CMP_EQ, ">=": VD_CMP_GE, "<=": V
 
 class vd_column(Structure):
     _fields_ = [("data", c_void_p), ("len", c_int64), ("dtype", c_int32), ("scale", c_int32), ("min", c_int64),
-                ("max", c_int64), ("has_minmax", c_int32), ("reserved", c_int32)]
+                ("max", c_int64), ("has_minmax", c_int32), ("flags", c_int32)]
 
 
 class vd_ctrl(Structure):
@@ -125,6 +126,9 @@ _sigs = {
                                   c_void_p, c_void_p, c_size_t, c_void_p]),
     "vd_merge_partials": (c_int32, [_P(vd_pipeline), _P(vd_column), c_int32, _P(vd_column), c_int32,
                                     _P(c_void_p), c_int32, c_void_p]),
+    "vd_group_fold_ws_bytes": (c_int32, [c_int64, c_int32, _P(c_size_t)]),
+    "vd_group_fold": (c_int32, [_P(vd_column), c_int32, c_int64, _P(vd_pred), c_int32, _P(vd_agg), c_int32,
+                                c_void_p, c_void_p, c_void_p, c_void_p, c_void_p, c_size_t, c_void_p]),
     "vd_last_launch_count": (c_int32, []),
     "vd_last_fragment": (ctypes.c_char_p, []),
     "vd_abi_struct_sizes": (c_int32, [_P(c_size_t), c_int32]),
@@ -205,8 +209,10 @@ def _stream(stream) -> Optional[int]:
     return stream if isinstance(stream, int) else stream.cuda_stream
 
 
-def column(t, minmax: Optional[Sequence[int]] = None, scale: int = 0, length: Optional[int] = None) -> vd_column:
-    """A vd_column view of a contiguous CUDA tensor (no copy)."""
+def column(t, minmax: Optional[Sequence[int]] = None, scale: int = 0, length: Optional[int] = None,
+           noeps: bool = False) -> vd_column:
+    """A vd_column view of a contiguous CUDA tensor (no copy).  noeps: the
+    caller has verified that no slot is epsilon (sets VD_COL_NOEPS)."""
     if not t.is_contiguous():
         raise VdError(VD_E_SHAPE, "column tensors must be contiguous")
     c = vd_column()
@@ -217,6 +223,8 @@ def column(t, minmax: Optional[Sequence[int]] = None, scale: int = 0, length: Op
     if minmax is not None:
         c.min, c.max = int(minmax[0]), int(minmax[1])
         c.has_minmax = 1
+    if noeps:
+        c.flags |= VD_COL_NOEPS
     c._keep = t  # the view keeps its tensor alive (the ABI struct holds a raw pointer)
     return c
 
@@ -367,6 +375,26 @@ def fold_max(vals, ctl=None, *, out, out_counts=None, out_nruns=None, ws=None, s
     _fold(_L.vd_fold_max, "vd_fold_max", vals, ctl, out, out_counts, out_nruns, ws, stream)
 
 
+def describe(t, scale: int = 0, stream=None) -> vd_column:
+    """a1 metadata for a device-resident column: min / max of
+    the non-epsilon values and VD_COL_NOEPS, computed on the device by the
+    library's own FoldMin / FoldMax (their per-run non-epsilon counts tell
+    whether any slot is epsilon).  Float columns get no metadata."""
+    import torch
+    c = column(t, scale=scale)
+    if c.dtype in (VD_F32, VD_F64) or t.numel() == 0:
+        return c
+    lo = torch.empty(1, dtype=t.dtype, device=t.device)
+    hi = torch.empty(1, dtype=t.dtype, device=t.device)
+    cnt = torch.empty(1, dtype=torch.int64, device=t.device)
+    fold_min(c, None, out=lo, out_counts=cnt, stream=stream)
+    fold_max(c, None, out=hi, stream=stream)
+    k = int(cnt.item())
+    if k == 0:
+        return c
+    return column(t, minmax=(int(lo.item()), int(hi.item())), scale=scale, noeps=(k == t.numel()))
+
+
 # ---- a4 gather / a5 scatter, partition -------------------------------------------------------
 def gather(src: vd_column, pos, n, bias, out, stream=None):
     _ok(_L.vd_gather(ctypes.byref(src), _ptr(pos), n, bias, _ptr(out), _stream(stream)), "vd_gather")
@@ -449,6 +477,51 @@ def pipeline(*, pred_: Optional[vd_pred] = None, sel_mode: int = VD_SEL_BRANCH, 
             p.aggs[i].f[j].col, p.aggs[i].f[j].a, p.aggs[i].f[j].b = f
     p.force_generic = int(force_generic)
     return p
+
+
+def aggs_array(aggs):
+    """A ctypes vd_agg[] from the pipeline() aggregate notation."""
+    return (vd_agg * max(1, len(aggs)))(*pipeline(aggs=aggs).aggs[:max(1, len(aggs))]) if aggs else None
+
+
+def group_fold_ws_bytes(domain: int, naggs: int) -> int:
+    b = c_size_t(0)
+    _ok(_L.vd_group_fold_ws_bytes(domain, naggs, ctypes.byref(b)), "vd_group_fold_ws_bytes")
+    return int(b.value)
+
+
+def group_fold(cols: Sequence[vd_column], n: int, key_col: int, aggs=(), pred_: Optional[vd_pred] = None, *,
+               out_keys, out_aggs, out_rows, out_ngroups, ws=None, stream=None):
+    """vd_group_fold (NEXT-4): grouped fold over the key column's min/max
+    domain; outputs are CUDA tensors (int64 keys / rows / ngroups[1], uint8
+    aggregate slots of 16 bytes x naggs per group)."""
+    k = cols[key_col]
+    if ws is None:
+        if not k.has_minmax:
+            raise VdError(VD_E_DOMAIN, "group_fold: key column without min/max")
+        ws = alloc_ws(group_fold_ws_bytes(k.max - k.min + 1, len(aggs)), out_keys.device)
+    arr = _cols_array(cols)
+    ag = aggs_array(aggs)
+    _ok(_L.vd_group_fold(arr, len(cols), n, ctypes.byref(pred_) if pred_ is not None else None, key_col, ag,
+                         len(aggs), out_keys.data_ptr(), _ptr(out_aggs), out_rows.data_ptr(), out_ngroups.data_ptr(),
+                         ws.data_ptr(), ws.numel(), _stream(stream)), "vd_group_fold")
+
+
+def decode_group_slots(buf: bytes, ngroups: int, naggs: int, float_aggs: Sequence[bool] = ()):
+    """[[agg values] per group] from vd_group_fold's 16-byte slots."""
+    import struct
+    out = []
+    for g in range(ngroups):
+        vals = []
+        for a in range(naggs):
+            off = (g * naggs + a) * 16
+            if a < len(float_aggs) and float_aggs[a]:
+                vals.append(struct.unpack_from("<d", buf, off)[0])
+            else:
+                lo, hi = struct.unpack_from("<Qq", buf, off)
+                vals.append(hi * (1 << 64) + lo)
+        out.append(vals)
+    return out
 
 
 def partials_bytes(plan: vd_pipeline) -> int:

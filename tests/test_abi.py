@@ -170,3 +170,39 @@ def test_row_layout_reading_fig14():
     assert vd.row_layout([vd.VD_I32, vd.VD_I32]) == ([0, 4], 8)
     with pytest.raises(vd.VdError):
         vd.row_layout([vd.VD_U8, vd.VD_F64, vd.VD_F64, vd.VD_F64, vd.VD_U8])
+
+
+def test_group_fold_host_validation():
+    """vd_group_fold (NEXT-4) validates before touching the device: the key's
+    min/max metadata sizes the table (VD_E_DOMAIN without, or beyond
+    VD_MAX_DOMAIN), integer SUMs must be provably exact (VD_E_OVERFLOW), the
+    workspace is checked (VD_E_WORKSPACE), and without a GPU the call fails
+    loudly (VD_E_CUDA: no CPU fallback)."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    L = vd._L
+
+    def col(dt, lo=None, hi=None):
+        c = vd.vd_column()
+        c.data, c.len, c.dtype = 256, 1000, dt
+        if lo is not None:
+            c.min, c.max, c.has_minmax = lo, hi, 1
+        return c
+
+    out = ctypes.c_void_p(4096)
+
+    def call(cols, aggs, ws=None, wsb=0):
+        arr = (vd.vd_column * len(cols))(*cols)
+        ag = vd.aggs_array(aggs)
+        return L.vd_group_fold(arr, len(cols), 1000, None, 0, ag, len(aggs), out, out, out, out, ws, wsb, None)
+
+    assert call([col(vd.VD_I64), col(vd.VD_I64, 0, 10)], [("count",)]) == vd.VD_E_DOMAIN
+    assert call([col(vd.VD_I64, 0, 2**40), col(vd.VD_I64, 0, 10)], [("count",)]) == vd.VD_E_DOMAIN
+    assert call([col(vd.VD_I64, 0, 99), col(vd.VD_I64, 0, 2**60)], [("sum", [1])]) == vd.VD_E_OVERFLOW
+    assert call([col(vd.VD_I64, 0, 99), col(vd.VD_I64)], [("sum", [1])]) == vd.VD_E_OVERFLOW
+    assert call([col(vd.VD_I64, 0, 99), col(vd.VD_F64)], [("min", [1])]) == vd.VD_E_UNSUPPORTED
+    assert call([col(vd.VD_I64, 0, 99), col(vd.VD_I64, 0, 10)], [("sum", [1]), ("count",)]) == vd.VD_E_WORKSPACE
+    need = vd.group_fold_ws_bytes(100, 2)
+    assert need >= 100 * 3 * 8
+    st = call([col(vd.VD_I64, 0, 99), col(vd.VD_I64, 0, 10)], [("sum", [1]), ("count",)], ctypes.c_void_p(1 << 20),
+              need)
+    assert st == vd.VD_E_CUDA

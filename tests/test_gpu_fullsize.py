@@ -33,15 +33,8 @@ def device_columns(names, n, sf, row0=0, table=gen.LINEITEM_COLS):
         gen.device(col, t.data_ptr(), n, row0, sf=sf)
         cols.append(t)
     torch.cuda.synchronize()
-    for t in cols:  # min/max metadata through the library's own folds (a1)
-        if t.dtype in (torch.float32, torch.float64):
-            views.append(vd.column(t))
-            continue
-        lo = torch.empty(1, dtype=t.dtype, device="cuda")
-        hi = torch.empty(1, dtype=t.dtype, device="cuda")
-        vd.fold_min(vd.column(t), None, out=lo)
-        vd.fold_max(vd.column(t), None, out=hi)
-        views.append(vd.column(t, minmax=(int(lo.item()), int(hi.item()))))
+    for t in cols:  # min/max + no-epsilon metadata through the library's own folds (a1)
+        views.append(vd.describe(t))
     return cols, views
 
 

@@ -356,7 +356,7 @@ def test_layout_transform_vs_interpreter(fields, n):
     vd.zip_rows([vd.column(c) for c in dcols], rows)
     outs = [torch.empty(max(n, 1), dtype=d.dtype, device="cuda") for d in dcols]
     vd.gather_rows(rows, m, dts, cuda_tensor(pos), n, 1, outs)
-    assert vd.last_launch_count() == 1
+    assert vd.last_launch_count() == (1 if n else 0)
     # row bytes: each field at its offset, padding zero
     rb = rows.cpu().numpy().reshape(m, stride)
     for c, o in zip(cols, offs):

@@ -309,6 +309,79 @@ def test_fkj_q9_vs_oracle(sel_mode, generic, n):
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
+@pytest.mark.parametrize("variant", ["fk_group_priv", "fk_group_priv_checked", "fk_group"])
+@pytest.mark.parametrize("n", [1023, 1024, 70001])
+def test_fkj_q9_fk_group_variants(variant, n):
+    """The Q9 FK grouped fold through each of its kernels: private slots with
+    the checks proven away (metadata with VD_COL_NOEPS), private slots with
+    per-row checks (no epsilon metadata), shared-memory atomics."""
+    import os
+    sf = 0.05
+    li = lineitem(sf, n)
+    part, supp = _dims(sf)
+    exp = oracle.fkj(1, li, part, supp)
+    keep, views = load([li[c] for c in plans.Q9_COLS])
+    dkeep, dviews = load([supp[c] for c in plans.Q9_DIMS])
+    if variant != "fk_group_priv":
+        for v in views + dviews:
+            v.flags = 0
+    plan = plans.q9()
+    if variant != "fk_group":
+        os.environ["VD_FKG_VARIANT"] = "priv"
+    try:
+        got = vd.decode_partials(run(plan, views, n, dviews, want=(variant,))[0], plan)
+    finally:
+        os.environ.pop("VD_FKG_VARIANT", None)
+    assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
+@pytest.mark.parametrize("variant", ["fk_group_priv_checked", "fk_group", "generic"])
+def test_fkj_q9_epsilon_vs_interpreter(variant):
+    """Q9 with epsilon everywhere, against the oracle's Voodoo program (Fig
+    10/11 shape): an epsilon or out-of-range l_suppkey gathers epsilon
+    (A11), an epsilon nation or ship date makes the key epsilon -- the row
+    has no group (A9, Partition drops it) -- and an epsilon l_extendedprice
+    or l_discount makes the row's revenue epsilon: skipped by the SUM (A5)
+    but the row still counts (COUNT(*) = FoldCount over the key)."""
+    import datetime
+    import os
+    sf = 0.05
+    n = 100003
+    li = lineitem(sf, n)
+    part, supp = _dims(sf)
+    rng = np.random.default_rng(11)
+    eps = {c: rng.random(n) < 0.01 for c in plans.Q9_COLS}
+    for c, e in eps.items():
+        li[c] = li[c].copy()
+        li[c][e] = {"i": -2**31 if li[c].dtype == np.int32 else -2**63}[li[c].dtype.kind]
+    oob = rng.random(n) < 0.005
+    li["l_suppkey"][oob & ~eps["l_suppkey"]] = len(supp["s_nationkey"]) + 5
+    nat = supp["s_nationkey"].copy()
+    enat = rng.random(len(nat)) < 0.02
+    nat[enat] = 0xFF
+    day0 = 8035
+    cal = np.array([(datetime.date(1970, 1, 1) + datetime.timedelta(days=day0 + i)).year for i in range(3000)])
+    p = oracle.Program()
+    for c in plans.Q9_COLS:
+        p.set("lineitem." + c, li[c], eps[c])
+    p.set("supplier.s_nationkey", nat, enat)
+    p.set("calendar.year", cal)
+    p.run(__import__("oracle.programs", fromlist=["x"]).FKJ_Q9.format(day0=day0)
+          + "rows := FoldCount(sc.g, sc.g)\no_rows := Gather(rows, gpos)\n")
+    keys = p.get("o_key")
+    exp = {k: (p.get("o_rev")[j] or 0, p.get("o_rows")[j]) for j, k in enumerate(keys) if k is not None}
+    keep, views = load([li[c] for c in plans.Q9_COLS])
+    dkeep, dviews = load([nat])
+    plan = plans.q9(force_generic=(variant == "generic"))
+    if variant == "fk_group_priv_checked":
+        os.environ["VD_FKG_VARIANT"] = "priv"
+    try:
+        got = vd.decode_partials(run(plan, views, n, dviews, want=(variant,))[0], plan)
+    finally:
+        os.environ.pop("VD_FKG_VARIANT", None)
+    assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
 def test_generic_min_max_and_float_products():
     """Generic fragment: MIN/MAX and float aggregates, grouped, with epsilon."""
     n = 200003

@@ -164,3 +164,27 @@ def test_fkj_q19_bruteforce_pandas():
     exp = {0: (rev, int(m.sum()))} if m.sum() else {}
     assert bf == exp
     assert m.sum() > 0  # the workload selects something at this size
+
+
+@pytest.mark.parametrize("sf", [0.002, 0.01])
+def test_q15_interpreter_bruteforce_pandas(sf):
+    """NEXT-4 pin: the Q15 revenue view grouped by l_suppkey (a large key
+    domain: every supplier is a group).  Brute force (sort + runs) ==
+    pandas groupby == the interpreter's Fig 10/11 program whose pivots
+    cover the key's min..max range."""
+    li = lineitem(sf)
+    d0, d1 = 9496, 9587
+    bf = oracle.q15(li, d0, d1)
+    m = (li["l_shipdate"] >= d0) & (li["l_shipdate"] < d1)
+    df = pd.DataFrame({"k": li["l_suppkey"][m],
+                       "rev": li["l_extendedprice"][m].astype(object) * (100 - li["l_discount"][m]).astype(object)})
+    g = df.groupby("k").agg(r=("rev", "sum"), c=("rev", "size"))
+    assert bf == {int(k): (int(r), int(c)) for k, (r, c) in zip(g.index, g.to_numpy())}
+    assert len(bf) > 0.5 * gen.supplier_rows(sf)  # high cardinality: most suppliers are groups
+    kmin, kmax = int(li["l_suppkey"].min()), int(li["l_suppkey"].max())
+    p = oracle.Program()
+    bind(p, "lineitem", li)
+    p.run(programs.Q15.format(d0m1=d0 - 1, d1=d1, kmin=kmin, D=kmax - kmin + 1))
+    keys = [k for k in p.get("o_key") if k is not None]
+    got = {k + kmin: (p.get("o_rev")[j], p.get("o_cnt")[j]) for j, k in enumerate(keys)}
+    assert got == bf
