@@ -168,7 +168,7 @@ vd_status vd_ctrl_runs(const vd_ctrl* ctrl, int64_t n, int64_t* nruns_host);
 
 /* Operator ids for vd_workspace_bytes. */
 typedef enum { VD_OP_SELECT = 0, VD_OP_FOLD = 1, VD_OP_SCATTER = 2, VD_OP_PIPELINE = 3, VD_OP_FOLD_SELECT = 4,
-               VD_OP_PARTITION = 5 } vd_op;
+               VD_OP_PARTITION = 5, VD_OP_FOLD_SCAN = 6 } vd_op;
 /* Scratch bytes needed by `op` over n input slots (out_len for SCATTER;
  * ngroups*naggs for PIPELINE is taken from `plan`, which may be NULL
  * otherwise). */
@@ -240,6 +240,17 @@ vd_status vd_fold_min(const vd_column* vals, const vd_ctrl* ctrl, void* out, int
                       int64_t* out_nruns_dev, void* ws, size_t ws_bytes, void* stream);
 vd_status vd_fold_max(const vd_column* vals, const vd_ctrl* ctrl, void* out, int64_t* out_counts,
                       int64_t* out_nruns_dev, void* ws, size_t ws_bytes, void* stream);
+
+/* FoldScan(.out, V1, .fold, .s) (Table 2): out[i] = sum of the
+ * non-epsilon vals[j] for j <= i in the same run of `ctrl` as i -- the
+ * prefix sum restarts at every run (inclusive, reading A27); an epsilon
+ * slot stays epsilon in out.  out has vals->len slots: integer input ->
+ * int64 (epsilon INT64_MIN; an i64 column needs min/max metadata proving
+ * |value| * len < 2^63, else VD_E_OVERFLOW), float input -> f64 (epsilon
+ * NaN; the association order is fixed per launch shape).
+ * ws: vd_workspace_bytes(VD_OP_FOLD_SCAN, len, ...). */
+vd_status vd_fold_scan(const vd_column* vals, const vd_ctrl* ctrl, void* out, void* ws, size_t ws_bytes,
+                       void* stream);
 
 /* ---------------------------------------------------------------------- */
 /* a4  Gather (Table 2; FK as position P:L452-456)              */

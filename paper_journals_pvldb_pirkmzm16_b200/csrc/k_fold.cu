@@ -18,6 +18,8 @@
 // Integer sums are exact 128-bit, float sums f64.
 #include <float.h>
 
+#include <cstring>
+
 #include "vd_common.cuh"
 #include "vd_internal.h"
 
@@ -447,6 +449,206 @@ cudaError_t launch_fold(FoldOp op, const vd_column& vals, const CtrlInfo& ci, vo
     case FOLD_COUNT: return fold_op<FOLD_COUNT>(vals, ci, starts, nstarts, out, out_counts, out_nruns, fws, s, nl);
     case FOLD_MIN: return fold_op<FOLD_MIN>(vals, ci, starts, nstarts, out, out_counts, out_nruns, fws, s, nl);
     default: return fold_op<FOLD_MAX>(vals, ci, starts, nstarts, out, out_counts, out_nruns, fws, s, nl);
+    }
+}
+
+// ============================================================================
+// FoldScan(.out, V1, .fold, .s) (Table 2): prefix sum of the values,
+// a new run of the control vector starting a new sum; inclusive, epsilon
+// slots stay epsilon and add nothing (reading A27).  One pass: tiles of
+// SCAN_T rows taken in order from an atomic counter; each thread scans 16
+// rows in registers, a CTA segmented scan (flag = "a run starts here")
+// joins threads, and a decoupled look-back over per-tile (flag, value) words
+// supplies the carry into the tile's first run.  A tile that contains a run
+// start publishes its inclusive prefix at once (the sum of its last run
+// does not depend on earlier tiles), so look-back chains stop there.
+// Integer input -> int64 (exactness proven on the host), float -> f64.
+// ============================================================================
+constexpr int FSC_THREADS = 256;
+constexpr int FSC_ITEMS = 16;
+constexpr int FSC_TILE = FSC_THREADS * FSC_ITEMS;
+
+struct FscStatus {
+    unsigned long long flag;  // 0 not ready, 1 aggregate ready, 2 inclusive prefix ready
+    unsigned long long agg;   // int64 or f64 bits; written once
+    unsigned long long pfx;   // written once, before flag = 2
+};
+
+template <typename A> __device__ __forceinline__ unsigned long long fsc_bits(A v);
+template <> __device__ __forceinline__ unsigned long long fsc_bits<int64_t>(int64_t v) { return (unsigned long long)v; }
+template <> __device__ __forceinline__ unsigned long long fsc_bits<double>(double v) {
+    return (unsigned long long)__double_as_longlong(v);
+}
+template <typename A> __device__ __forceinline__ A fsc_val(unsigned long long b);
+template <> __device__ __forceinline__ int64_t fsc_val<int64_t>(unsigned long long b) { return (int64_t)b; }
+template <> __device__ __forceinline__ double fsc_val<double>(unsigned long long b) {
+    return __longlong_as_double((long long)b);
+}
+
+__device__ __forceinline__ void fsc_publish(FscStatus* st, unsigned long long flag, unsigned long long val) {
+    if (flag == 2ull) st->pfx = val;
+    else st->agg = val;
+    __threadfence();
+    asm volatile("st.release.gpu.global.u64 [%0], %1;" ::"l"(&st->flag), "l"(flag) : "memory");
+}
+
+template <typename T, typename A>
+__global__ void __launch_bounds__(FSC_THREADS) k_fold_scan(const T* __restrict__ v, int64_t n, RidSrc rs,
+                                                           A* __restrict__ out, FscStatus* __restrict__ status,
+                                                           unsigned long long* __restrict__ tile_ctr) {
+    __shared__ int64_t s_tile;
+    __shared__ int s_wf[FSC_THREADS / 32];
+    __shared__ A s_ws[FSC_THREADS / 32];
+    __shared__ A s_carry;
+    const int t = threadIdx.x, lane = t & 31, warp = t >> 5;
+    if (t == 0) s_tile = (int64_t)atomicAdd(tile_ctr, 1ull);
+    __syncthreads();
+    const int64_t tile = s_tile;
+    const int64_t row0 = tile * FSC_TILE + (int64_t)t * FSC_ITEMS;
+
+    // thread-local inclusive segmented scan
+    A y[FSC_ITEMS];
+    unsigned hm = 0, em = 0;
+    A run = 0;
+#pragma unroll
+    for (int j = 0; j < FSC_ITEMS; ++j) {
+        const int64_t i = row0 + j;
+        bool h = false;
+        if (i < n) {
+            if (rs.cls == RUNS_ONE) h = (i == 0);
+            else if (rs.cls == RUNS_FIXED) h = (i % rs.R) == 0;
+            else h = (i == 0) || (rs.value(i) != rs.value(i - 1));
+        }
+        if (h) run = 0;
+        T x = i < n ? __ldg(v + i) : Eps<T>::value();
+        const bool e = Eps<T>::is(x);
+        if (!e) run += (A)x;
+        y[j] = run;
+        hm |= (h ? 1u : 0u) << j;
+        em |= (e ? 1u : 0u) << j;
+    }
+    // CTA segmented inclusive scan of (flag, sum) over threads
+    int f = hm != 0;
+    A sum = run;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        const int fp = __shfl_up_sync(VD_FULL, f, o);
+        const A sp = __shfl_up_sync(VD_FULL, sum, o);
+        if (lane >= o) {
+            if (!f) sum += sp;
+            f |= fp;
+        }
+    }
+    if (lane == 31) { s_wf[warp] = f; s_ws[warp] = sum; }
+    __syncthreads();
+    if (warp == 0) {
+        int wf = lane < FSC_THREADS / 32 ? s_wf[lane] : 0;
+        A wsum = lane < FSC_THREADS / 32 ? s_ws[lane] : (A)0;
+#pragma unroll
+        for (int o = 1; o < FSC_THREADS / 32; o <<= 1) {
+            const int fp = __shfl_up_sync(VD_FULL, wf, o);
+            const A sp = __shfl_up_sync(VD_FULL, wsum, o);
+            if (lane >= o) {
+                if (!wf) wsum += sp;
+                wf |= fp;
+            }
+        }
+        // tile aggregate = inclusive value of the last warp
+        const int tf = __shfl_sync(VD_FULL, wf, FSC_THREADS / 32 - 1);
+        const A tsum = __shfl_sync(VD_FULL, wsum, FSC_THREADS / 32 - 1);
+        if (lane < FSC_THREADS / 32) { s_wf[lane] = wf; s_ws[lane] = wsum; }  // inclusive per warp
+        // look-back: the carry into this tile's first run
+        A carry = 0;
+        if (tile > 0) {
+            if (lane == 0 && tf) fsc_publish(&status[tile], 2ull, fsc_bits<A>(tsum));
+            else if (lane == 0) fsc_publish(&status[tile], 1ull, fsc_bits<A>(tsum));
+            int64_t end = tile - 1;
+            for (;;) {
+                const int64_t idx = end - lane;
+                unsigned long long fl = 2ull, vb = fsc_bits<A>((A)0);
+                if (idx >= 0) {
+                    do {
+                        asm volatile("ld.acquire.gpu.global.u64 %0, [%1];" : "=l"(fl) : "l"(&status[idx].flag) : "memory");
+                    } while (fl == 0);
+                    vb = fl == 2ull ? __ldcg(&status[idx].pfx) : __ldcg(&status[idx].agg);
+                }
+                const unsigned pm = __ballot_sync(VD_FULL, fl == 2ull);
+                const int stop = pm ? (__ffs(pm) - 1) : 31;
+                A c = lane <= stop ? fsc_val<A>(vb) : (A)0;
+                // fixed-order reduction (deterministic for floats)
+#pragma unroll
+                for (int o = 16; o > 0; o >>= 1) c += __shfl_xor_sync(VD_FULL, c, o);
+                carry += c;
+                if (pm) break;
+                end -= 32;
+            }
+            if (lane == 0 && !tf) fsc_publish(&status[tile], 2ull, fsc_bits<A>(carry + tsum));
+        } else if (lane == 0) {
+            fsc_publish(&status[0], 2ull, fsc_bits<A>(tsum));
+        }
+        if (lane == 0) s_carry = carry;
+    }
+    __syncthreads();
+    // exclusive (flag, sum) before this thread, then the tile carry
+    int pf = 0;
+    A ps = 0;
+    {
+        const int fp = __shfl_up_sync(VD_FULL, f, 1);
+        const A sp = __shfl_up_sync(VD_FULL, sum, 1);
+        if (lane > 0) { pf = fp; ps = sp; }
+        if (warp > 0) {
+            // prepend the previous warps' inclusive value
+            const int wf = s_wf[warp - 1];
+            const A wsv = s_ws[warp - 1];
+            if (!pf) { ps += wsv; pf = wf; }
+        }
+        if (!pf) ps += s_carry;
+    }
+#pragma unroll
+    for (int j = 0; j < FSC_ITEMS; ++j) {
+        const int64_t i = row0 + j;
+        if (i >= n) break;
+        const bool before_head = (hm & ((2u << j) - 1u)) == 0;  // no run start in rows 0..j of this thread
+        A r = y[j] + (before_head ? ps : (A)0);
+        if ((em >> j) & 1u) {
+            out[i] = fsc_val<A>(sizeof(A) == 8 && !IsFloat<A>::value ? 0x8000000000000000ull : 0x7ff8000000000000ull);
+        } else {
+            out[i] = r;
+        }
+    }
+}
+
+size_t fold_scan_ws_bytes(int64_t n) {
+    const int64_t ntiles = (n + FSC_TILE - 1) / FSC_TILE;
+    return 256 + (((size_t)ntiles * sizeof(FscStatus) + 255) & ~(size_t)255);
+}
+
+template <typename T, typename A>
+static cudaError_t fold_scan_typed(const vd_column& vals, const CtrlInfo& ci, void* out, void* ws, cudaStream_t s,
+                                   int* nl) {
+    const int64_t n = vals.len;
+    const int64_t ntiles = (n + FSC_TILE - 1) / FSC_TILE;
+    if (ntiles == 0) return cudaSuccess;
+    cudaError_t e = cudaMemsetAsync(ws, 0, fold_scan_ws_bytes(n), s);
+    if (e != cudaSuccess) return e;
+    RidSrc rs;
+    std::memset(&rs, 0, sizeof(rs));
+    rs.cls = ci.cls; rs.R = ci.R; rs.mat = ci.mat; rs.dt = ci.mat_dtype;
+    rs.from = ci.from; rs.num = ci.num; rs.den = ci.den; rs.cap = ci.cap;
+    k_fold_scan<T, A><<<(unsigned)ntiles, FSC_THREADS, 0, s>>>((const T*)vals.data, n, rs, (A*)out,
+                                                               (FscStatus*)((char*)ws + 256),
+                                                               (unsigned long long*)ws);
+    ++*nl;
+    return cudaGetLastError();
+}
+
+cudaError_t launch_fold_scan(const vd_column& vals, const CtrlInfo& ci, void* out, void* ws, cudaStream_t s, int* nl) {
+    switch (vals.dtype) {
+    case VD_U8: return fold_scan_typed<uint8_t, int64_t>(vals, ci, out, ws, s, nl);
+    case VD_I32: return fold_scan_typed<int32_t, int64_t>(vals, ci, out, ws, s, nl);
+    case VD_I64: return fold_scan_typed<int64_t, int64_t>(vals, ci, out, ws, s, nl);
+    case VD_F32: return fold_scan_typed<float, double>(vals, ci, out, ws, s, nl);
+    default: return fold_scan_typed<double, double>(vals, ci, out, ws, s, nl);
     }
 }
 

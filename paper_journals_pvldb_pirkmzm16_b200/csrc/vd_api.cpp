@@ -318,6 +318,7 @@ vd_status vd_workspace_bytes(int32_t op, int64_t n, const vd_ctrl* ctrl, const s
     case VD_OP_FOLD: *bytes = fold_total_ws(n, ci); return VD_OK;
     case VD_OP_SCATTER: *bytes = scatter_ws_bytes(n); return VD_OK;
     case VD_OP_PARTITION: *bytes = partition_ws_bytes(n, 1024); return VD_OK;
+    case VD_OP_FOLD_SCAN: *bytes = fold_scan_ws_bytes(n); return VD_OK;
     case VD_OP_PIPELINE:
         if (!plan) return VD_E_NULL;
         if (plan->ngroups < 1 || plan->ngroups > VD_MAX_GROUPS || plan->naggs < 0 || plan->naggs > VD_MAX_AGGS)
@@ -414,6 +415,30 @@ vd_status vd_fold_min(const vd_column* vals, const vd_ctrl* ctrl, void* out, int
 vd_status vd_fold_max(const vd_column* vals, const vd_ctrl* ctrl, void* out, int64_t* out_counts, int64_t* out_nruns,
                       void* ws, size_t ws_bytes, void* stream) {
     return fold_entry(FOLD_MAX, vals, ctrl, out, out_counts, out_nruns, ws, ws_bytes, stream);
+}
+
+vd_status vd_fold_scan(const vd_column* vals, const vd_ctrl* ctrl, void* out, void* ws, size_t ws_bytes, void* stream) {
+    reset_launches();
+    vd_status st = check_col(vals, 0, "fold_scan");
+    if (st != VD_OK) return st;
+    if (vals->len > 0 && (!out || !vals->data)) { set_error("fold_scan: NULL out / data"); return VD_E_NULL; }
+    if (vals->len > INT32_MAX) { set_error("fold_scan: n must be < 2^31"); return VD_E_SHAPE; }
+    if (vals->dtype == VD_I64) {
+        // int64 running sums: |value| * n must stay below 2^63 (metadata)
+        const double b = std::max(std::fabs((double)vals->min), std::fabs((double)vals->max)) * (double)vals->len;
+        if (!vals->has_minmax || b >= 9.2e18) {
+            set_error("fold_scan: min/max metadata cannot prove int64 running sums exact");
+            return VD_E_OVERFLOW;
+        }
+    }
+    CtrlInfo ci;
+    if ((st = classify_ctrl(ctrl, vals->len, &ci)) != VD_OK) return st;
+    if ((st = check_ws(ws, ws_bytes, fold_scan_ws_bytes(vals->len))) != VD_OK) return st;
+    if ((st = check_device()) != VD_OK) return st;
+    int nl = 0;
+    st = cuda_status(launch_fold_scan(*vals, ci, out, ws, (cudaStream_t)stream, &nl));
+    count_launches(nl);
+    return st;
 }
 
 vd_status vd_gather_multi(const vd_column* srcs, int32_t nsrc, const int32_t* pos, int64_t n, int64_t bias,

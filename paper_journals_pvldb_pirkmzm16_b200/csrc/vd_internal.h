@@ -76,6 +76,9 @@ size_t fold_ws_bytes(int64_t n);
 cudaError_t launch_fold(FoldOp op, const vd_column& vals, const CtrlInfo& ci, void* out, int64_t* out_counts,
                         int64_t* out_nruns, void* ws, size_t ws_bytes, cudaStream_t s, int* nlaunch);
 
+size_t fold_scan_ws_bytes(int64_t n);
+cudaError_t launch_fold_scan(const vd_column& vals, const CtrlInfo& ci, void* out, void* ws, cudaStream_t s, int* nl);
+
 // k_gather.cu
 cudaError_t launch_gather(const vd_column* srcs, int nsrc, const int32_t* pos, int64_t n, int64_t bias,
                           void* const* outs, cudaStream_t s, int* nlaunch);

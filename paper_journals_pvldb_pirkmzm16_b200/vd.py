@@ -31,7 +31,7 @@ VD_OK, VD_E_NULL, VD_E_DTYPE, VD_E_SHAPE, VD_E_CTRL, VD_E_DOMAIN, VD_E_OVERFLOW,
 VD_U8, VD_I32, VD_I64, VD_F32, VD_F64 = range(5)
 VD_CMP_GT, VD_CMP_LT, VD_CMP_EQ, VD_CMP_GE, VD_CMP_LE, VD_CMP_NE, VD_CMP_IN = range(7)
 VD_SEL_BRANCH, VD_SEL_PREDICATED, VD_SEL_PREDICATED_LOOKUP = 0, 1, 2
-VD_OP_SELECT, VD_OP_FOLD, VD_OP_SCATTER, VD_OP_PIPELINE, VD_OP_FOLD_SELECT, VD_OP_PARTITION = range(6)
+VD_OP_SELECT, VD_OP_FOLD, VD_OP_SCATTER, VD_OP_PIPELINE, VD_OP_FOLD_SELECT, VD_OP_PARTITION, VD_OP_FOLD_SCAN = range(7)
 VD_AGG_SUM, VD_AGG_COUNT, VD_AGG_MIN, VD_AGG_MAX = range(4)
 VD_SCATTER_UNIQUE = 1
 VD_COL_NOEPS = 1
@@ -112,6 +112,7 @@ _sigs = {
                               c_void_p]),
     "vd_fold_max": (c_int32, [_P(vd_column), _P(vd_ctrl), c_void_p, c_void_p, c_void_p, c_void_p, c_size_t,
                               c_void_p]),
+    "vd_fold_scan": (c_int32, [_P(vd_column), _P(vd_ctrl), c_void_p, c_void_p, c_size_t, c_void_p]),
     "vd_gather": (c_int32, [_P(vd_column), c_void_p, c_int64, c_int64, c_void_p, c_void_p]),
     "vd_gather_multi": (c_int32, [_P(vd_column), c_int32, c_void_p, c_int64, c_int64, _P(c_void_p), c_void_p]),
     "vd_row_layout": (c_int32, [_P(c_int32), c_int32, _P(c_int32), _P(c_int32)]),
@@ -373,6 +374,16 @@ def fold_min(vals, ctl=None, *, out, out_counts=None, out_nruns=None, ws=None, s
 
 def fold_max(vals, ctl=None, *, out, out_counts=None, out_nruns=None, ws=None, stream=None):
     _fold(_L.vd_fold_max, "vd_fold_max", vals, ctl, out, out_counts, out_nruns, ws, stream)
+
+
+def fold_scan(vals, ctl=None, *, out, ws=None, stream=None):
+    """vd_fold_scan: per-run inclusive prefix sums into `out` (int64 or
+    float64 CUDA tensor of vals.len slots)."""
+    if ws is None:
+        ws = alloc_ws(workspace_bytes(VD_OP_FOLD_SCAN, vals.len, ctl), out.device)
+    c = ctypes.byref(ctl) if ctl is not None else None
+    _ok(_L.vd_fold_scan(ctypes.byref(vals), c, _ptr(out), ws.data_ptr(), ws.numel(), _stream(stream)),
+        "vd_fold_scan")
 
 
 def describe(t, scale: int = 0, stream=None) -> vd_column:

@@ -206,3 +206,21 @@ def test_group_fold_host_validation():
     st = call([col(vd.VD_I64, 0, 99), col(vd.VD_I64, 0, 10)], [("sum", [1]), ("count",)], ctypes.c_void_p(1 << 20),
               need)
     assert st == vd.VD_E_CUDA
+
+
+def test_fold_scan_host_validation():
+    """vd_fold_scan: an i64 column needs min/max metadata proving its running
+    sums fit int64 (VD_E_OVERFLOW otherwise); workspace checked; no GPU ->
+    VD_E_CUDA."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    L = vd._L
+    c = vd.vd_column()
+    c.data, c.len, c.dtype = 256, 1000, vd.VD_I64
+    out = ctypes.c_void_p(4096)
+    assert L.vd_fold_scan(ctypes.byref(c), None, out, None, 0, None) == vd.VD_E_OVERFLOW
+    c.min, c.max, c.has_minmax = -2**60, 2**60, 1
+    assert L.vd_fold_scan(ctypes.byref(c), None, out, None, 0, None) == vd.VD_E_OVERFLOW
+    c.min, c.max = -2**40, 2**40
+    assert L.vd_fold_scan(ctypes.byref(c), None, out, None, 0, None) == vd.VD_E_WORKSPACE
+    need = vd.workspace_bytes(vd.VD_OP_FOLD_SCAN, 1000)
+    assert L.vd_fold_scan(ctypes.byref(c), None, out, ctypes.c_void_p(1 << 20), need, None) == vd.VD_E_CUDA

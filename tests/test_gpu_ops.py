@@ -300,6 +300,51 @@ def test_hierarchical_fold_fig3_fig4_on_gpu():
     assert tot == i128_from_bytes(o3.cpu().numpy().tobytes(), 0) == int(a.astype(object).sum())
 
 
+@pytest.mark.parametrize("dtype", ["u8", "i32", "i64", "f32", "f64"])
+@pytest.mark.parametrize("kind", CTRLS)
+@pytest.mark.parametrize("n", [0, 1, 4095, 4096, 70001])
+def test_fold_scan_vs_interpreter(dtype, kind, n):
+    """FoldScan (Table 2; reading A27): per-run inclusive prefix sums
+    restarting at each run, epsilon slots stay epsilon, against the oracle's
+    FoldScan -- across tile boundaries (4096-row tiles), runs shorter and
+    longer than a tile, irregular virtual and materialized controls.  Integer
+    exact; float within 1e-9 relative of the long-double oracle (positive
+    data: no cancellation)."""
+    rng = np.random.default_rng(abs(hash((dtype, str(kind), n))) % 2**32)
+    if dtype == "u8":
+        a = rng.integers(0, 250, n).astype(np.uint8)
+    elif dtype == "i32":
+        a = rng.integers(-2**31 + 1, 2**31 - 1, n).astype(np.int32)
+    elif dtype == "i64":
+        a = rng.integers(-2**40, 2**40, n).astype(np.int64)
+    elif dtype == "f32":
+        a = rng.random(n).astype(np.float32)
+    else:
+        a = rng.random(n) * 1e6
+    a, m = with_eps(a, 0.05, 3)
+    cvals, c, keep = make_ctrl(kind, n, seed=9)
+    dv = cuda_tensor(a)
+    col = vd.column(dv, minmax=(-2**40, 2**40) if dtype == "i64" else None)
+    isf = a.dtype.kind == "f"
+    out = torch.full((max(n, 1),), 7, dtype=torch.float64 if isf else torch.int64, device="cuda")
+    vd.fold_scan(col, c, out=out)
+    assert vd.last_launch_count() == (1 if n else 0)
+    if n == 0:
+        return
+    vals = a.astype(np.float64) if isf else a.astype(np.int64)
+    p = oracle.run("r := FoldScan(k, v)", k=cvals, v=(vals, m))
+    o = out[:n].cpu().numpy()
+    if isf:
+        ve, re_, e = p.get_float_exact("r")
+        assert np.array_equal(np.isnan(o), e)
+        ref = ve[~e] + re_[~e]
+        assert np.all(np.abs(o[~e] - ref) <= REL * np.abs(ref) + 1e-300)
+    else:
+        ev, ee = p.get_arrays("r")
+        assert np.array_equal(o == -2**63, ee)
+        assert np.array_equal(o[~ee], np.asarray(ev)[~ee].astype(np.int64))
+
+
 # ---------------------------------------------------------------------------
 # a4 gather, a5 scatter / partition
 # ---------------------------------------------------------------------------
