@@ -410,8 +410,17 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
     int32_t* st = s_stage + warp * (BM_CHUNK + BM_CHUNK / 32);
+    // the next chunk's bitmap word and offset are loaded one iteration ahead,
+    // so their round trip overlaps this chunk's decode and stores
+    uint32_t w_nx = gw < nchunks ? __ldcs(&bits[gw * 32 + lane]) : 0u;
+    int64_t base_nx = gw < nchunks ? __ldcs(&offs[gw]) : 0;
     for (int64_t c = gw; c < nchunks; c += nw) {
-        const uint32_t w = bits[c * 32 + lane];
+        const uint32_t w = w_nx;
+        const int64_t base = base_nx;
+        if (c + nw < nchunks) {
+            w_nx = __ldcs(&bits[(c + nw) * 32 + lane]);
+            base_nx = __ldcs(&offs[c + nw]);
+        }
         const int pc = __popc(w);
         int incl = pc;
 #pragma unroll
@@ -442,8 +451,7 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
             }
         }
         __syncwarp();
-        const int64_t base = offs[c];
-        for (int k = lane; k < total; k += 32) out[base + k] = st[k + (k >> 5)];
+        for (int k = lane; k < total; k += 32) __stcs(&out[base + k], st[k + (k >> 5)]);
         __syncwarp();
     }
 }
