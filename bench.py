@@ -36,6 +36,7 @@ METRIC = "rows/s and achieved HBM GB/s (% of peak) for TPC-H Q1/Q6 at 1/2/4/8 B2
 # column each query reads, once.
 BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "q19": 4 + 3 * 8 + 1 + 1,
                  "q9": 4 + 4 + 2 * 8, "fkjsel": 4 + 4}
+L2_CAP_BYTES_PER_CLK = 6300  # B300_MICROARCH.md "LTS throughput cap" (full chip)
 
 
 def parse():
@@ -355,7 +356,31 @@ def main():
 
     peak, peak_kind = hbm_peak()
     bpr = BYTES_PER_ROW[w]
-    achieved = n * bpr / (kernel_ms * 1e-3) / 1e9  # per GPU, dominant-kernel duration
+    alg_bytes = n * bpr
+    extra = {}
+    if w == "fkjsel":
+        # reading A33: a lookup into a table larger than L2 (16 Mi x 8 B =
+        # 128 MiB) moves one 64-byte HBM block; branching and predicated-lookup
+        # plans look up the qualifying rows only (the lookup plan sends the
+        # rest to the hot slot 0), predicated aggregation looks up every row
+        sel_rows = int(next(iter(result.values()))[-1]) if result else 0
+        looked_up = n if args.sel_mode == "predicated" else sel_rows // max(world, 1)
+        alg_bytes = n * bpr + 64 * looked_up
+        extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64}
+    elif w in ("q9", "q19"):
+        # the dimension lookups hit L2 (supplier 1 MB; part 120 MB at SF100):
+        # the second bound is L2 slice throughput, one 32-byte sector per
+        # lookup on top of the streamed sectors
+        nlook = n if w == "q9" else None
+        if nlook is not None:
+            sectors = n * bpr / 32 + nlook
+            clk_ghz = (clk or {}).get("sm_mhz") or 1965.0
+            cap = L2_CAP_BYTES_PER_CLK * clk_ghz / 1e3 / 32  # sectors per ns
+            ach = sectors / (kernel_ms * 1e6)
+            extra = {"l2": {"bound": "l2", "sectors_per_row": bpr / 32 + 1, "achieved": ach, "peak": cap,
+                            "unit": "sectors/ns", "frac": ach / cap,
+                            "peak_kind": "guide: B300-measured LTS cap 6300 B/clk x SM clock (B300_MICROARCH.md)"}}
+    achieved = alg_bytes / (kernel_ms * 1e-3) / 1e9  # per GPU, dominant-kernel duration
     rows_per_s = n_total / (ms_per_step * 1e-3)
     line = {
         "metric": METRIC,
@@ -384,9 +409,9 @@ def main():
         "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                      "frac": achieved / peak, "peak_kind": peak_kind,
                      "traffic": ncu_traffic(f"fkjsel_s{args.selectivity:g}_{args.sel_mode}" if w == "fkjsel" else w),
-                     "bytes_per_row": bpr,
+                     "bytes_per_row": alg_bytes / n if n else bpr,
                      "kernel": "k_pipe_q1+k_q1_remap" if w == "q1" and not args.generic else "vd_run_pipeline",
-                     "kernel_ms": kernel_ms},
+                     "kernel_ms": kernel_ms, **extra},
         "clocks": clk,
         "e2e": e2e,
         "gpu_launches": launches_per_step * steps,

@@ -328,7 +328,7 @@ __device__ __forceinline__ uint32_t spread8(uint32_t x) {  // bit k -> bit 4k
     return x;
 }
 
-template <typename T, bool ALIGNED>
+template <typename T, bool ALIGNED, bool IVL>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNED> fl, int64_t n,
                                                              uint32_t* __restrict__ bits,
                                                              int32_t* __restrict__ counts, int64_t nchunks) {
@@ -337,18 +337,37 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNE
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
     uint32_t* bal = s_bal[warp];
+    // chunks entirely inside the column (all but the last): no per-row
+    // bounds checks, and the interval form of the term (IVL, decided on the
+    // host) as two compares with no epsilon / operator dispatch
+    const int64_t nfull = ALIGNED ? n / BM_CHUNK : 0;
     for (int64_t c = gw; c < nchunks; c += nw) {
-        typename TermFlags<T, ALIGNED>::Raw raw[8];
+        if (c < nfull) {
+            T v[8][4];
 #pragma unroll
-        for (int q = 0; q < 8; ++q) fl.load(c * BM_CHUNK + q * 128 + lane * 4, n, raw[q]);
+            for (int q = 0; q < 8; ++q) Vec4Load<T>::ld(fl.p + c * BM_CHUNK + q * 128 + lane * 4, v[q]);
 #pragma unroll
-        for (int q = 0; q < 8; ++q) {
-            bool f[4];
-            fl.eval(raw[q], c * BM_CHUNK + q * 128 + lane * 4, n, f);
+            for (int q = 0; q < 8; ++q) {
 #pragma unroll
-            for (int j = 0; j < 4; ++j) {
-                const uint32_t b = __ballot_sync(VD_FULL, f[j]);
-                if (lane == 0) bal[q * 4 + j] = b;  // bit L <-> row q*128 + 4L + j
+                for (int j = 0; j < 4; ++j) {
+                    const bool f = IVL ? (v[q][j] >= fl.lo && v[q][j] <= fl.hi) : fl.test(v[q][j]);
+                    const uint32_t b = __ballot_sync(VD_FULL, f);
+                    if (lane == 0) bal[q * 4 + j] = b;  // bit L <-> row q*128 + 4L + j
+                }
+            }
+        } else {
+            typename TermFlags<T, ALIGNED>::Raw raw[8];
+#pragma unroll
+            for (int q = 0; q < 8; ++q) fl.load(c * BM_CHUNK + q * 128 + lane * 4, n, raw[q]);
+#pragma unroll
+            for (int q = 0; q < 8; ++q) {
+                bool f[4];
+                fl.eval(raw[q], c * BM_CHUNK + q * 128 + lane * 4, n, f);
+#pragma unroll
+                for (int j = 0; j < 4; ++j) {
+                    const uint32_t b = __ballot_sync(VD_FULL, f[j]);
+                    if (lane == 0) bal[q * 4 + j] = b;
+                }
             }
         }
         __syncwarp();
@@ -481,8 +500,15 @@ static size_t bm_ws_bytes(int64_t n) {
     int64_t nc = (n + BM_CHUNK - 1) / BM_CHUNK;
     return al256((size_t)nc * 32 * 4) + al256((size_t)nc * 4) + al256((size_t)nc * 8) + scan_ws_bytes(nc) + 256;
 }
-static int bm_grid(int64_t nchunks) {
-    int64_t g = (int64_t)num_sms() * 8;
+// One resident wave: blocks per SM from the kernel's occupancy (registers,
+// shared memory), times the SM count -- a grid-stride loop over a grid
+// larger than one wave leaves its last partial wave running alone.
+template <class K>
+static int bm_grid(K kern, int64_t nchunks) {
+    int per_sm = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, BM_THREADS, 0) != cudaSuccess || per_sm < 1)
+        per_sm = 1;
+    int64_t g = (int64_t)num_sms() * per_sm;
     int64_t need = (nchunks * 32 + BM_THREADS - 1) / BM_THREADS;
     if (g > need) g = need;
     return (int)(g < 1 ? 1 : g);
@@ -493,13 +519,13 @@ static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t*
                                      void* ws, cudaStream_t s, int* nl) {
     BmLayout L = bm_layout(n, ws);
     if (L.nchunks == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
-    launch_bits(L, bm_grid(L.nchunks));
+    launch_bits(L);
     ++*nl;
     cudaError_t e = cudaGetLastError();
     if (e != cudaSuccess) return e;
     if ((e = launch_scan_i32(L.counts, L.nchunks, L.offs, L.scan_ws, s, nl)) != cudaSuccess) return e;
     k_sel_total<<<1, 1, 0, s>>>(L.offs, L.counts, L.nchunks, out_count);
-    k_sel_write<MODE><<<bm_grid(L.nchunks), BM_THREADS, 0, s>>>(L.bits, L.offs, L.nchunks, out_pos);
+    k_sel_write<MODE><<<bm_grid(k_sel_write<MODE>, L.nchunks), BM_THREADS, 0, s>>>(L.bits, L.offs, L.nchunks, out_pos);
     *nl += 2;
     return cudaGetLastError();
 }
@@ -589,16 +615,17 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         return run_select_bitmap<MODE>(
-            [&](const BmLayout& L, int grid) {
-                k_sel_bits_vec<T, true><<<grid, BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+            [&](const BmLayout& L) {
+                if (ivl) k_sel_bits_vec<T, true, true><<<bm_grid(k_sel_bits_vec<T, true, true>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+                else k_sel_bits_vec<T, true, false><<<bm_grid(k_sel_bits_vec<T, true, false>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
             },
             n, out_pos, out_count, ws, s, nl);
     }
     TermFlags<T, false> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
     if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
     return run_select_bitmap<MODE>(
-        [&](const BmLayout& L, int grid) {
-            k_sel_bits_vec<T, false><<<grid, BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+        [&](const BmLayout& L) {
+            k_sel_bits_vec<T, false, false><<<bm_grid(k_sel_bits_vec<T, false, false>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
         },
         n, out_pos, out_count, ws, s, nl);
 }
@@ -620,8 +647,8 @@ static cudaError_t select_mode(const DevCols& cols, const DevPred& pred, int64_t
     GenericFlags g{pred, cols};
     if (use_lookback()) return run_select<MODE>(g, n, out_pos, out_count, ws, s, nl);
     return run_select_bitmap<MODE>(
-        [&](const BmLayout& L, int grid) {
-            k_sel_bits_bal<GenericFlags><<<grid, BM_THREADS, 0, s>>>(g, n, L.bits, L.counts, L.nchunks);
+        [&](const BmLayout& L) {
+            k_sel_bits_bal<GenericFlags><<<bm_grid(k_sel_bits_bal<GenericFlags>, L.nchunks), BM_THREADS, 0, s>>>(g, n, L.bits, L.counts, L.nchunks);
         },
         n, out_pos, out_count, ws, s, nl);
 }
@@ -637,8 +664,8 @@ cudaError_t launch_select_heads(const CtrlInfo& ci, int64_t n, int32_t* out_pos,
     HeadFlags h{ci.mat, ci.mat_dtype, ci.from, ci.num, ci.den, ci.cap};
     if (use_lookback()) return run_select<0>(h, n, out_pos, out_count, ws, s, nl);
     return run_select_bitmap<0>(
-        [&](const BmLayout& L, int grid) {
-            k_sel_bits_bal<HeadFlags><<<grid, BM_THREADS, 0, s>>>(h, n, L.bits, L.counts, L.nchunks);
+        [&](const BmLayout& L) {
+            k_sel_bits_bal<HeadFlags><<<bm_grid(k_sel_bits_bal<HeadFlags>, L.nchunks), BM_THREADS, 0, s>>>(h, n, L.bits, L.counts, L.nchunks);
         },
         n, out_pos, out_count, ws, s, nl);
 }

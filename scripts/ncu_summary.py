@@ -35,6 +35,9 @@ KEYS = [
     "smsp__average_warps_issue_stalled_math_pipe_throttle_per_issue_active.ratio",
     "smsp__average_warps_issue_stalled_no_instruction_per_issue_active.ratio",
     "l1tex__data_pipe_lsu_wavefronts_mem_shared.sum",
+    "lts__t_sectors.sum", "lts__t_sectors.sum.per_second", "lts__t_sectors_srcunit_tex_op_read.sum",
+    "lts__throughput.avg.pct_of_peak_sustained_elapsed", "lts__t_sector_hit_rate.pct",
+    "l1tex__t_sector_hit_rate.pct",
 ]
 
 SCALE = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "Tbyte": 1e12}
