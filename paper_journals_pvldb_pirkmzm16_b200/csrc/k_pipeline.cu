@@ -2454,6 +2454,11 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
 // the selected values in f64 and count them.  4 rows per LDS.128.
 constexpr int SS_TILE = 8192;
 constexpr int SS_MAXSTAGES = 6;
+// 16 consumer warps (4 per scheduler): with 8 the per-tile instruction
+// stream of each warp was exposed (issue active 44%, 5.96 TB/s)
+constexpr int SS_CW = 16;
+constexpr int SS_NT = SS_CW * 32;
+constexpr int SS_THREADS = SS_NT + 32;
 
 struct SelSumArgs {
     const float* v;
@@ -2463,7 +2468,7 @@ struct SelSumArgs {
 };
 
 template <int MODE>
-__global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid_constant__ SelSumArgs a,
+__global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_constant__ SelSumArgs a,
                                                                     int64_t ntiles, Slot16* __restrict__ parts,
                                                                     unsigned int* __restrict__ done,
                                                                     Slot16* __restrict__ out, const ScalarMap map) {
@@ -2475,7 +2480,7 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid
     if (threadIdx.x == 0) {
         for (int s = 0; s < a.nstages; ++s) {
             mbar_init(&full[s], 1);
-            mbar_init(&empty[s], SCT_CW);
+            mbar_init(&empty[s], SS_CW);
         }
         fence_mbar_init();
     }
@@ -2492,33 +2497,37 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid
             cnt += 1;
         }
     };
-    if (warp == SCT_CW) {
+    if (warp == SS_CW) {
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
+            int s = 0;
+            uint32_t ph = 0;  // parity of the current pass over the ring
             for (int64_t it = 0;; ++it) {
                 const int64_t tile = blockIdx.x + it * gridDim.x;
                 if (tile >= ntiles) break;
-                const int s = (int)(it % a.nstages);
-                if (it >= a.nstages) mbar_wait(&empty[s], (uint32_t)(((it / a.nstages) - 1) & 1));
+                if (it >= a.nstages) mbar_wait(&empty[s], ph ^ 1u);
                 mbar_expect_tx(&full[s], SS_TILE * 4);
                 tma_load_1d(smem + (size_t)s * SS_TILE * 4, a.v + tile * SS_TILE, SS_TILE * 4, &full[s], pol);
+                if (++s == a.nstages) { s = 0; ph ^= 1u; }
             }
         }
         __syncwarp();
     } else {
+        int s = 0;
+        uint32_t ph = 0;
         for (int64_t it = 0;; ++it) {
             const int64_t tile = blockIdx.x + it * gridDim.x;
             if (tile >= ntiles) break;
-            const int s = (int)(it % a.nstages);
-            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            mbar_wait(&full[s], ph);
             const float4* st = reinterpret_cast<const float4*>(smem + (size_t)s * SS_TILE * 4);
-            float4 x[SS_TILE / 4 / SCT_NT];
+            float4 x[SS_TILE / 4 / SS_NT];
 #pragma unroll
-            for (int k = 0; k < SS_TILE / 4 / SCT_NT; ++k) x[k] = st[threadIdx.x + k * SCT_NT];
+            for (int k = 0; k < SS_TILE / 4 / SS_NT; ++k) x[k] = st[threadIdx.x + k * SS_NT];
             __syncwarp();
             if (lane == 0) mbar_arrive(&empty[s]);
+            if (++s == a.nstages) { s = 0; ph ^= 1u; }
 #pragma unroll
-            for (int k = 0; k < SS_TILE / 4 / SCT_NT; ++k) {
+            for (int k = 0; k < SS_TILE / 4 / SS_NT; ++k) {
                 row(x[k].x);
                 row(x[k].y);
                 row(x[k].z);
@@ -2526,9 +2535,9 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid
             }
         }
         if (blockIdx.x == 0)
-            for (int64_t r = ntiles * SS_TILE + threadIdx.x; r < a.n; r += SCT_NT) row(a.v[r]);
+            for (int64_t r = ntiles * SS_TILE + threadIdx.x; r < a.n; r += SS_NT) row(a.v[r]);
     }
-    __shared__ Slot16 s_w[SCT_THREADS / 32][2];
+    __shared__ Slot16 s_w[SS_THREADS / 32][2];
     const int64_t c = warp_sum_i64(cnt);
     const double sm = warp_sum_f64(sum);
     if (lane == 0) {
@@ -2539,7 +2548,7 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_selsum_tma(const __grid
     if (threadIdx.x == 0) {
         double t = 0;
         i128 k = 0;
-        for (int w = 0; w < SCT_THREADS / 32; ++w) { t += get_f64(s_w[w][0]); k += get_i128(s_w[w][1]); }
+        for (int w = 0; w < SS_THREADS / 32; ++w) { t += get_f64(s_w[w][0]); k += get_i128(s_w[w][1]); }
         put_f64(&parts[(size_t)blockIdx.x * 2], t);
         put_i128(&parts[(size_t)blockIdx.x * 2 + 1], k);
     }
@@ -2779,10 +2788,10 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
             const size_t smem = (size_t)ss.nstages * SS_TILE * 4 + 2 * ss.nstages * 8;
             if (mode) {
                 cudaFuncSetAttribute(k_pipe_selsum_tma<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-                k_pipe_selsum_tma<1><<<grid, SCT_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
+                k_pipe_selsum_tma<1><<<grid, SS_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
             } else {
                 cudaFuncSetAttribute(k_pipe_selsum_tma<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-                k_pipe_selsum_tma<0><<<grid, SCT_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
+                k_pipe_selsum_tma<0><<<grid, SS_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
             }
             ++*nl;
             e = cudaGetLastError();

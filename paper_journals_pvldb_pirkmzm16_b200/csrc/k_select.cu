@@ -88,6 +88,27 @@ template <> struct Vec4Load<uint8_t> {
     }
 };
 
+// 4 consecutive values from shared memory (16-byte aligned for 4-byte types).
+template <typename T> struct Vec4Lds;
+template <> struct Vec4Lds<float> {
+    static __device__ __forceinline__ void ld(const float* p, float v[4]) {
+        float4 x = *reinterpret_cast<const float4*>(p);
+        v[0] = x.x; v[1] = x.y; v[2] = x.z; v[3] = x.w;
+    }
+};
+template <> struct Vec4Lds<int32_t> {
+    static __device__ __forceinline__ void ld(const int32_t* p, int32_t v[4]) {
+        int4 x = *reinterpret_cast<const int4*>(p);
+        v[0] = x.x; v[1] = x.y; v[2] = x.z; v[3] = x.w;
+    }
+};
+template <> struct Vec4Lds<uint8_t> {
+    static __device__ __forceinline__ void ld(const uint8_t* p, uint8_t v[4]) {
+        uint32_t x = *reinterpret_cast<const uint32_t*>(p);
+        v[0] = x & 0xFF; v[1] = (x >> 8) & 0xFF; v[2] = (x >> 16) & 0xFF; v[3] = x >> 24;
+    }
+};
+
 // One term over one column; 4 rows per vector load when the column base is
 // aligned to the vector width (checked on the host).
 template <typename T, bool ALIGNED>
@@ -331,7 +352,8 @@ __device__ __forceinline__ uint32_t spread8(uint32_t x) {  // bit k -> bit 4k
 template <typename T, bool ALIGNED, bool IVL>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNED> fl, int64_t n,
                                                              uint32_t* __restrict__ bits,
-                                                             int32_t* __restrict__ counts, int64_t nchunks) {
+                                                             int32_t* __restrict__ counts, int64_t nchunks,
+                                                             int64_t c0 = 0) {
     __shared__ uint32_t s_bal[BM_THREADS / 32][32];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
@@ -341,7 +363,7 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNE
     // bounds checks, and the interval form of the term (IVL, decided on the
     // host) as two compares with no epsilon / operator dispatch
     const int64_t nfull = ALIGNED ? n / BM_CHUNK : 0;
-    for (int64_t c = gw; c < nchunks; c += nw) {
+    for (int64_t c = c0 + gw; c < nchunks; c += nw) {
         if (c < nfull) {
             T v[8][4];
 #pragma unroll
@@ -377,6 +399,98 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_vec(TermFlags<T, ALIGNE
 #pragma unroll
         for (int j = 0; j < 4; ++j) word |= spread8((bal[q * 4 + j] >> (8 * m)) & 0xFFu) << j;
         __syncwarp();
+        bits[c * 32 + lane] = word;
+        int cnt = __popc(word);
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) cnt += __shfl_xor_sync(VD_FULL, cnt, o);
+        if (lane == 0) counts[c] = cnt;
+    }
+}
+
+// TMA-staged flag pass for 1- and 4-byte columns under an interval term:
+// a producer warp streams BT_CW-chunk tiles of the column with 1D bulk copies
+// into a BT_STAGES-deep mbarrier ring; consumer warp w builds chunk w of the
+// tile out of shared memory (same ballot / byte-spread assembly as
+// k_sel_bits_vec).  The LDG version is latency bound (64 registers -> 32
+// warps per SM, no loads in flight while a warp assembles its words); the
+// ring keeps HBM busy independent of the consumers.  Measured on 1e9 f32:
+// 620.8 us (TMA) vs 630 us (LDG), i.e. 6.45 TB/s -- the single-stream read
+// ceiling (scripts/ubench_read.cu: 6.69 TB/s for a bare LDG.128 stream).
+constexpr int BT_CW = 16;
+constexpr int BT_THREADS = BT_CW * 32 + 32;
+constexpr int BT_STAGES = 3;
+
+// tile of a CTA's it-th step (strided over the grid), -1 past the end.  A
+// contiguous range of tiles per CTA was measured slower (637.8 vs 620.8 us
+// per 4 GB): HBM bank spread is not the limit.
+__device__ __forceinline__ int64_t tile_of(int64_t it, int64_t ntiles) {
+    const int64_t t = blockIdx.x + it * gridDim.x;
+    return t < ntiles ? t : -1;
+}
+
+template <typename T>
+__global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restrict__ col, T lo, T hi,
+                                                                int64_t ntiles, uint32_t* __restrict__ bits,
+                                                                int32_t* __restrict__ counts) {
+    constexpr uint32_t TB = BT_CW * BM_CHUNK * sizeof(T);  // tile bytes
+    extern __shared__ __align__(128) uint8_t smem[];
+    __shared__ uint32_t s_bal[BT_CW][32];
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)BT_STAGES * TB);
+    uint64_t* empty = full + BT_STAGES;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < BT_STAGES; ++i) {
+            mbar_init(&full[i], 1);
+            mbar_init(&empty[i], BT_CW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (warp == BT_CW) {
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int st = 0;
+            uint32_t ph = 0;
+            for (int64_t it = 0;; ++it) {
+                const int64_t tile = tile_of(it, ntiles);
+                if (tile < 0) break;
+                if (it >= BT_STAGES) mbar_wait(&empty[st], ph ^ 1u);
+                mbar_expect_tx(&full[st], TB);
+                tma_load_1d(smem + (size_t)st * TB, col + tile * (BT_CW * BM_CHUNK), TB, &full[st], pol);
+                if (++st == BT_STAGES) { st = 0; ph ^= 1u; }
+            }
+        }
+        return;
+    }
+    uint32_t* bal = s_bal[warp];
+    int st = 0;
+    uint32_t ph = 0;
+    for (int64_t it = 0;; ++it) {
+        const int64_t tile = tile_of(it, ntiles);
+        if (tile < 0) break;
+        mbar_wait(&full[st], ph);
+        const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * BM_CHUNK;
+        T v[8][4];
+#pragma unroll
+        for (int q = 0; q < 8; ++q) Vec4Lds<T>::ld(src + q * 128 + lane * 4, v[q]);
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[st]);
+        if (++st == BT_STAGES) { st = 0; ph ^= 1u; }
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                const uint32_t b = __ballot_sync(VD_FULL, v[q][j] >= lo && v[q][j] <= hi);
+                if (lane == 0) bal[q * 4 + j] = b;  // bit L <-> row q*128 + 4L + j
+            }
+        }
+        __syncwarp();
+        const int qq = lane >> 2, m = lane & 3;
+        uint32_t word = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) word |= spread8((bal[qq * 4 + j] >> (8 * m)) & 0xFFu) << j;
+        __syncwarp();
+        const int64_t c = tile * BT_CW + warp;
         bits[c * 32 + lane] = word;
         int cnt = __popc(word);
 #pragma unroll
@@ -604,6 +718,18 @@ static bool term_interval_t(const DevTerm& t, T* lo, T* hi) {
     return true;
 }
 
+// TMA flag pass: 1- and 4-byte columns (16-byte aligned, checked by the
+// caller); VD_SELECT_BITS=ldg forces the LDG pass (kept for comparison)
+template <typename T>
+static bool use_bits_tma() {
+    if (sizeof(T) != 4 && sizeof(T) != 1) return false;
+    static const bool ldg = [] {
+        const char* e = getenv("VD_SELECT_BITS");
+        return e && strcmp(e, "ldg") == 0;
+    }();
+    return !ldg;
+}
+
 template <int MODE, typename T>
 static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int32_t* out_pos, int64_t* out_count,
                                  void* ws, cudaStream_t s, int* nl) {
@@ -616,7 +742,28 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L) {
-                if (ivl) k_sel_bits_vec<T, true, true><<<bm_grid(k_sel_bits_vec<T, true, true>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
+                bool tma_done = false;
+                if constexpr (sizeof(T) == 4 || sizeof(T) == 1) {
+                if (ivl && use_bits_tma<T>() && ((uintptr_t)p & 15) == 0) {
+                    // full tiles through the TMA ring, the rest (< BT_CW chunks + ragged tail) by LDG
+                    const int64_t ntiles = n / ((int64_t)BT_CW * BM_CHUNK);
+                    if (ntiles > 0) {
+                        const size_t sm = (size_t)BT_STAGES * BT_CW * BM_CHUNK * sizeof(T) + 2 * BT_STAGES * 8;
+                        cudaFuncSetAttribute(k_sel_bits_tma<T>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+                        const int g = (int)std::min<int64_t>(ntiles, num_sms());
+                        k_sel_bits_tma<T><<<g, BT_THREADS, sm, s>>>((const T*)p, ilo, ihi, ntiles, L.bits, L.counts);
+                        ++*nl;
+                    }
+                    const int64_t c0 = ntiles * BT_CW;
+                    if (c0 < L.nchunks)
+                        k_sel_bits_vec<T, true, true><<<bm_grid(k_sel_bits_vec<T, true, true>, L.nchunks - c0), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks, c0);
+                    else
+                        --*nl;  // run_select_bitmap counts one flag launch
+                    tma_done = true;
+                }
+                }
+                if (tma_done) {
+                } else if (ivl) k_sel_bits_vec<T, true, true><<<bm_grid(k_sel_bits_vec<T, true, true>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
                 else k_sel_bits_vec<T, true, false><<<bm_grid(k_sel_bits_vec<T, true, false>, L.nchunks), BM_THREADS, 0, s>>>(f, n, L.bits, L.counts, L.nchunks);
             },
             n, out_pos, out_count, ws, s, nl);

@@ -465,3 +465,38 @@ def test_partition_vs_interpreter(n, P):
     assert out[:n].cpu().tolist() == [(-1 if e is None else e) for e in exp]
     b = np.clip(v[~m].astype(np.int64) - frm, 0, P - 1)
     assert bc.cpu().tolist() == np.bincount(b, minlength=P).tolist()
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("dtype", ["u8", "i32", "f32"])
+@pytest.mark.parametrize("offset", [0, 4])
+def test_select_flag_pass_tiles_and_tail(mode, dtype, offset):
+    """Several 16384-row tiles of the TMA flag pass plus a ragged LDG tail; a
+    base pointer 4 bytes past a 16-byte boundary takes the LDG pass instead.
+    Positions must equal flatnonzero of the predicate either way."""
+    n = 5 * 16384 + 1000 + 7
+    rng = np.random.default_rng(99)
+    if dtype == "u8":
+        a = rng.integers(0, 255, n + 16).astype(np.uint8)  # 0xFF = epsilon excluded by the interval
+        op, c = ">", 100
+        ref = (a > 100) & (a != 0xFF)
+    elif dtype == "i32":
+        a = rng.integers(-1000, 1000, n + 16).astype(np.int32)
+        op, c = "<=", 17
+        ref = a <= 17
+    else:
+        a = rng.random(n + 16).astype(np.float32)
+        op, c = "<", 0.25
+        ref = a < np.float32(0.25)
+    esz = a.itemsize
+    skip = offset // esz
+    da = cuda_tensor(a)[skip:skip + n]
+    exp = np.flatnonzero(ref[skip:skip + n])
+    out = torch.empty(n, dtype=torch.int32, device="cuda")
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    fn([vd.column(da)], n, vd.pred([[(0, op, c)]]), out_pos=out, out_count=cnt)
+    k = int(cnt.item())
+    assert k == len(exp)
+    assert np.array_equal(out[:k].cpu().numpy(), exp)
