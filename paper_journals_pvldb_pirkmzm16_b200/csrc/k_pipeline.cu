@@ -1351,6 +1351,219 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
 }
 
 // ============================================================================
+// Late-materialisation fragment (branching scalar plans, Fig 15/16 "branching"
+// strategy): only the LEAD columns -- the
+// columns of predicate terms common to every conjunction whose conjunction
+// is an interval (u8: any terms, checked value by value on the host; i32:
+// comparisons) -- stream densely (one 128-bit load per 16 rows per u8
+// column, four per i32 column).  Rows that pass are compacted per warp
+// (popc prefix over the lanes) into a shared-memory queue and folded 32 at a
+// time, every lane busy: the rest of the predicate, the FK gathers and the
+// aggregate inputs are loaded for those rows only (late loads, reading A31).
+// A dense TMA fragment moves every byte of every column; this one moves the
+// lead bytes plus the 64-byte blocks that hold a qualifying row.
+// ============================================================================
+struct LateLead {
+    const uint8_t* c8[2];
+    uint32_t lo8[2], hi8[2];  // interval bounds replicated into the 4 bytes
+    const int32_t* c32;
+    int32_t lo32, hi32;       // lo32 > INT32_MIN: epsilon never passes
+    // references (bit c: base column c, bit ncols + g: gather g) read by the
+    // rest of the predicate / by the aggregates; FK columns of the gathers
+    // included, so that each group of loads is issued at once
+    uint32_t pref, aref;
+};
+
+// A lead-qualified row: the predicate's columns and lookups are loaded in
+// two rounds (base columns, then the dimension lookups they address), all
+// loads of a round in flight together; the aggregate inputs are loaded only
+// when the row qualifies (late materialisation).
+__device__ __forceinline__ void late_load(const GfArgs& a, uint32_t want, uint32_t have, int64_t row, Val* v) {
+#pragma unroll
+    for (int c = 0; c < GF_MAXCOLS; ++c)
+        if (c < a.ncols && ((want & ~have) >> c & 1u)) v[c] = fetch_typed(a.col[c], a.dt[c], row);
+#pragma unroll
+    for (int g = 0; g < VD_MAX_GATHERS; ++g) {
+        const int r = a.ncols + g;
+        if (g < a.ngathers && ((want & ~have) >> r & 1u)) {
+            const Val fk = v[a.g_fk[g]];
+            const int64_t p = fk.i - a.g_bias[g];
+            if (fk.eps || p < 0 || p >= a.g_len[g]) {
+                v[r].eps = true;
+                v[r].isf = false;
+                v[r].i = 0;
+                v[r].f = 0;
+            } else {
+                v[r] = fetch_typed(a.g_p[g], a.g_dt[g], p);
+            }
+        }
+    }
+}
+
+__device__ __forceinline__ bool late_pred(const GfArgs& a, const Val* v) {
+    for (int k = 0; k < a.ncommon; ++k)
+        if (!term_true(a.common[k], v[a.common[k].col])) return false;
+    if (a.pred.nconj == 0) return true;
+    for (int c = 0; c < a.pred.nconj; ++c) {
+        bool ok = true;
+        for (int k = 0; k < a.pred.nterms[c] && ok; ++k) ok = term_true(a.pred.t[c][k], v[a.pred.t[c][k].col]);
+        if (ok) return true;
+    }
+    return false;
+}
+constexpr int LT_THREADS = 256;
+constexpr int LT_QCAP = 32 + 16 * 32;  // < 32 left over + one 16-row step of every lane
+
+// 16 u8 rows (one 128-bit word) against [lo, hi] per byte -> 16-bit mask
+__device__ __forceinline__ uint32_t lt_mask_u8(int4 v, uint32_t lo4, uint32_t hi4) {
+    const uint32_t w[4] = {(uint32_t)v.x, (uint32_t)v.y, (uint32_t)v.z, (uint32_t)v.w};
+    uint32_t m = 0;
+#pragma unroll
+    for (int i = 0; i < 4; ++i) {
+        const uint32_t r = __vcmpgeu4(w[i], lo4) & __vcmpleu4(w[i], hi4);  // 0xFF per passing byte
+        m |= (((r & 0x01010101u) * 0x01020408u) >> 24) << (4 * i);         // byte k -> bit k
+    }
+    return m;
+}
+
+template <int N8, bool I32>
+__global__ void __launch_bounds__(LT_THREADS) k_pipe_late(const __grid_constant__ GfArgs a,
+                                                         const __grid_constant__ LateLead ld,
+                                                         Slot16* __restrict__ parts, unsigned int* __restrict__ done,
+                                                         Slot16* __restrict__ out) {
+    __shared__ int32_t s_q[LT_THREADS / 32][LT_QCAP];
+    __shared__ int64_t s_acc[LT_THREADS / 32][VD_MAX_AGGS + 1];
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int NA = a.naggs;
+    int32_t* q_ = s_q[warp];
+    int cnt = 0;  // warp-uniform queue depth
+    int64_t racc[VD_MAX_AGGS + 1];
+#pragma unroll
+    for (int g = 0; g <= VD_MAX_AGGS; ++g) racc[g] = 0;
+    // the rest of the predicate and the aggregate inputs of one lead-qualified row
+    auto fold_row = [&](int64_t row) {
+        Val v[GF_MAXCOLS + VD_MAX_GATHERS];
+        const uint32_t pb = ld.pref & ((1u << a.ncols) - 1);
+        late_load(a, pb, 0, row, v);               // round 1: base columns of the predicate (+ FKs)
+        late_load(a, ld.pref & ~pb, pb, row, v);   // round 2: the lookups they address
+        if (!late_pred(a, v)) return;
+        const uint32_t ab = ld.aref & ((1u << a.ncols) - 1);
+        late_load(a, ab, ld.pref, row, v);
+        late_load(a, ld.aref & ~ab, ld.pref | ab, row, v);
+#pragma unroll
+        for (int g = 0; g < VD_MAX_AGGS; ++g) {
+            if (g >= NA) break;
+            int64_t pr = 1;
+            if (a.a_kind[g] != VD_AGG_COUNT) {
+                bool e = false;
+                for (int f = 0; f < a.a_nf[g]; ++f) {
+                    int64_t x = 0;
+                    if (a.a_col[g][f] >= 0) {
+                        const Val& u = v[a.a_col[g][f]];
+                        e |= u.eps;
+                        x = u.i;
+                    }
+                    pr *= a.a_a[g][f] + a.a_b[g][f] * x;
+                }
+                if (e) pr = 0;  // an epsilon input is skipped by the fold (A5)
+            }
+            racc[g] += pr;
+        }
+        racc[VD_MAX_AGGS] += 1;
+    };
+    auto drain = [&](int k) {  // fold the top k (<= 32) queued rows
+        __syncwarp();
+        if (lane < k) fold_row(q_[cnt - k + lane]);
+        cnt -= k;
+        __syncwarp();
+    };
+    const int64_t nq = a.n / 16;
+    const int64_t wstride = (int64_t)gridDim.x * LT_THREADS;
+    for (int64_t q0 = (int64_t)blockIdx.x * LT_THREADS + warp * 32; q0 < nq; q0 += wstride) {
+        const int64_t q = q0 + lane;
+        uint32_t m = 0;
+        if (q < nq) {
+            m = 0xFFFFu;
+#pragma unroll
+            for (int j = 0; j < N8; ++j) m &= lt_mask_u8(ld_stream16(ld.c8[j] + 16 * q), ld.lo8[j], ld.hi8[j]);
+            if (I32) {
+#pragma unroll
+                for (int k = 0; k < 4; ++k) {
+                    const int4 v = ld_stream16(ld.c32 + 16 * q + 4 * k);
+                    const int32_t x[4] = {v.x, v.y, v.z, v.w};
+#pragma unroll
+                    for (int j = 0; j < 4; ++j)
+                        if (x[j] < ld.lo32 || x[j] > ld.hi32) m &= ~(1u << (4 * k + j));
+                }
+            }
+        }
+        // compaction: the lanes' qualifying rows, in row order, onto the warp's queue
+        const int pc = __popc(m);
+        int incl = pc;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const int u = __shfl_up_sync(VD_FULL, incl, o);
+            if (lane >= o) incl += u;
+        }
+        int at = cnt + incl - pc;
+        while (m) {
+            q_[at++] = (int32_t)(16 * q + (__ffs(m) - 1));
+            m &= m - 1;
+        }
+        cnt += __shfl_sync(VD_FULL, incl, 31);
+        while (cnt >= 32) drain(32);
+    }
+    if (cnt > 0) drain(cnt);
+    // ragged tail (< 16 rows): warp 0 of block 0, one row per lane
+    if (blockIdx.x == 0 && warp == 0) {
+        const int64_t row = nq * 16 + lane;
+        if (row < a.n) {
+            bool ok = true;
+#pragma unroll
+            for (int j = 0; j < N8; ++j) {
+                const uint32_t x = ld.c8[j][row];
+                ok = ok && x >= (ld.lo8[j] & 0xFFu) && x <= (ld.hi8[j] & 0xFFu);
+            }
+            if (I32) ok = ok && ld.c32[row] >= ld.lo32 && ld.c32[row] <= ld.hi32;
+            if (ok) fold_row(row);
+        }
+    }
+    // fold: warp sums (int64, bounded on the host) -> CTA (int128) -> last CTA
+#pragma unroll
+    for (int g = 0; g <= VD_MAX_AGGS; ++g) {
+        const int64_t t = warp_sum_i64(racc[g]);
+        if (lane == 0) s_acc[warp][g] = t;
+    }
+    __syncthreads();
+    const int NS = NA + 1;
+    if (threadIdx.x < NS) {
+        const int g = threadIdx.x < NA ? threadIdx.x : VD_MAX_AGGS;
+        i128 t = 0;
+        for (int w = 0; w < LT_THREADS / 32; ++w) t += (i128)s_acc[w][g];
+        put_i128(&parts[(size_t)blockIdx.x * NS + threadIdx.x], t);
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x < NS) {
+        i128 t = 0;
+        for (unsigned b = 0; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * NS + threadIdx.x].lo);
+            x.hi = __ldcg(&parts[(size_t)b * NS + threadIdx.x].hi);
+            t += get_i128(x);
+        }
+        put_i128(&out[threadIdx.x], t);
+    }
+}
+
+// ============================================================================
 // FK grouped-fold fragment (Q9 shape): key = (dim[fk - bias] - subA) * mA +
 // (f(kb) - subB) * mB with f = calendar year (shared-memory table) or
 // identity, value = X * (a + b * Y) (32x32->64 IMAD.WIDE when proven narrow),
@@ -2969,8 +3182,14 @@ static vd_status try_fkg(const vd_pipeline* p, const vd_column* cols, int ncols,
                          2 * GF_MAXSTAGES * 8;
     const size_t budget = 200 * 1024;
     if (fixed + 2 * SB > budget) return VD_OK;
+    // a 2-stage ring (96 KB in flight per SM) is enough to keep HBM busy; the
+    // fragment is bound by L2 sector throughput, and deeper rings (4 stages)
+    // measured slower: 3.43 vs 3.20 ms at SF100 (streamed sectors queue ahead
+    // of the dimension lookups).  VD_FKG_STAGES overrides (2..budget).
     int ns = (int)((budget - fixed) / SB);
-    A.nstages = ns > GF_MAXSTAGES ? GF_MAXSTAGES : ns;
+    ns = ns > GF_MAXSTAGES ? GF_MAXSTAGES : ns;
+    A.nstages = 2;
+    if (const char* sv = getenv("VD_FKG_STAGES")) A.nstages = std::max(2, std::min(ns, atoi(sv)));
     const size_t smem = fixed + (size_t)A.nstages * SB;
     unsigned int* dn = (unsigned int*)ws;
     Slot16* parts = (Slot16*)((char*)ws + 256);
@@ -3263,8 +3482,30 @@ static vd_status try_star(const vd_pipeline* p, const vd_column* cols, int ncols
 }
 
 // ---- gather-fold matching -------------------------------------------------------
+// VD_LATE: "off" disables the late-materialisation fragment, "force" also
+// tries it before the dense scalar fragment (plans without gathers: Q6)
+static int late_policy() {
+    const char* e = getenv("VD_LATE");
+    if (e && strcmp(e, "off") == 0) return 0;
+    if (e && strcmp(e, "force") == 0) return 2;
+    return 1;
+}
+
+static bool host_cmp_int(int cmp, int64_t x, int64_t c) {  // = cmp_int (vd_pred.cuh)
+    switch (cmp) {
+    case VD_CMP_GT: return x > c;
+    case VD_CMP_LT: return x < c;
+    case VD_CMP_EQ: return x == c;
+    case VD_CMP_GE: return x >= c;
+    case VD_CMP_LE: return x <= c;
+    case VD_CMP_NE: return x != c;
+    case VD_CMP_IN: return (uint64_t)x < 64ull && (((uint64_t)c >> (uint64_t)x) & 1ull);
+    default: return false;
+    }
+}
+
 static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
-                        void* out, void* ws, cudaStream_t s, int* nl, bool* done) {
+                        void* out, void* ws, cudaStream_t s, int* nl, bool* done, bool late_only = false) {
     *done = false;
     const char* var = getenv("VD_GF_VARIANT");
     if (var && strcmp(var, "off") == 0) return VD_OK;
@@ -3400,6 +3641,98 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         if (mx * rows_per_warp >= 9.0e18) return VD_OK;
     }
     A.n = n;
+    if (late_only) {
+        // lead columns: base columns of hoisted terms whose conjunction is an
+        // interval (u8: checked value by value, epsilon 0xFF never passes;
+        // i32: comparisons only, epsilon INT32_MIN never passes)
+        const int lmode = p->sel_mode == VD_SEL_BRANCH ? 0 : 1;
+        // the warp queues hold int32 row numbers
+        if (p->ngroups != 1 || lmode != 0 || p->nkeyparts != 0 || n <= 0 || n >= INT32_MAX) return VD_OK;
+        LateLead L;
+        std::memset(&L, 0, sizeof(L));
+        int n8 = 0;
+        bool i32 = false;
+        bool lead[GF_MAXCOLS] = {};
+        for (int k = 0; k < A.ncommon; ++k) {
+            const int c = A.common[k].col;
+            if (c >= ncols || lead[c]) continue;
+            if (cols[c].dtype == VD_U8 && n8 < 2) {
+                bool pass[256];
+                int lo = 256, hi = -1;
+                for (int x = 0; x < 256; ++x) {
+                    bool ok = x != 0xFF;
+                    for (int h = 0; h < A.ncommon && ok; ++h)
+                        if (A.common[h].col == c) ok = host_cmp_int(A.common[h].cmp, x, A.common[h].iv);
+                    pass[x] = ok;
+                    if (ok) { lo = std::min(lo, x); hi = std::max(hi, x); }
+                }
+                bool ivl = true;
+                for (int x = lo; x <= hi && ivl; ++x) ivl = pass[x];
+                if (!ivl) continue;
+                if (hi < lo) { lo = 1; hi = 0; }  // nothing passes
+                L.c8[n8] = (const uint8_t*)cols[c].data;
+                L.lo8[n8] = 0x01010101u * (uint32_t)lo;
+                L.hi8[n8] = 0x01010101u * (uint32_t)hi;
+                ++n8;
+                lead[c] = true;
+            } else if (cols[c].dtype == VD_I32 && !i32) {
+                int64_t lo = (int64_t)INT32_MIN + 1, hi = INT32_MAX;
+                bool ivl = true;
+                for (int h = 0; h < A.ncommon && ivl; ++h) {
+                    if (A.common[h].col != c) continue;
+                    const int64_t v = A.common[h].iv;
+                    switch (A.common[h].cmp) {
+                    case VD_CMP_GT: lo = std::max(lo, v + 1); break;
+                    case VD_CMP_GE: lo = std::max(lo, v); break;
+                    case VD_CMP_LT: hi = std::min(hi, v - 1); break;
+                    case VD_CMP_LE: hi = std::min(hi, v); break;
+                    case VD_CMP_EQ: lo = std::max(lo, v); hi = std::min(hi, v); break;
+                    default: ivl = false;
+                    }
+                }
+                if (!ivl) continue;
+                if (lo > hi) { lo = 1; hi = 0; }
+                L.c32 = (const int32_t*)cols[c].data;
+                L.lo32 = (int32_t)lo;
+                L.hi32 = (int32_t)hi;
+                i32 = true;
+                lead[c] = true;
+            }
+        }
+        if (n8 == 0 && !i32) return VD_OK;
+        int nc = 0;  // the lead intervals replace the hoisted terms on their columns
+        for (int k = 0; k < A.ncommon; ++k)
+            if (!lead[A.common[k].col]) A.common[nc++] = A.common[k];
+        A.ncommon = nc;
+        // referenced columns (gathers: also their FK column)
+        auto ref = [&](uint32_t& m, int c) {
+            m |= 1u << c;
+            if (c >= ncols) m |= 1u << A.g_fk[c - ncols];
+        };
+        for (int k = 0; k < A.ncommon; ++k) ref(L.pref, A.common[k].col);
+        for (int c = 0; c < A.pred.nconj; ++c)
+            for (int k = 0; k < A.pred.nterms[c]; ++k) ref(L.pref, A.pred.t[c][k].col);
+        for (int g = 0; g < A.naggs; ++g)
+            if (A.a_kind[g] != VD_AGG_COUNT)
+                for (int f = 0; f < A.a_nf[g]; ++f)
+                    if (A.a_col[g][f] >= 0) ref(L.aref, A.a_col[g][f]);
+        const int grid = grid_persistent(4);  // the pipeline workspace holds 4 x SMs partial slots
+        unsigned int* dn = (unsigned int*)ws;
+        Slot16* parts = (Slot16*)((char*)ws + 256);
+        cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+#define LT_GO(N8_, I32_) k_pipe_late<N8_, I32_><<<grid, LT_THREADS, 0, s>>>(A, L, parts, dn, (Slot16*)out)
+        if (n8 == 2) { if (i32) LT_GO(2, true); else LT_GO(2, false); }
+        else if (n8 == 1) { if (i32) LT_GO(1, true); else LT_GO(1, false); }
+        else LT_GO(0, true);
+#undef LT_GO
+        ++*nl;
+        e = cudaGetLastError();
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+        set_fragment("late");
+        *done = true;
+        return VD_OK;
+    }
     // shared memory: ring + warp slots + staging + calendar + barriers
     const int NS = (int)p->ngroups * (p->naggs + 1);
     size_t fixed = (size_t)GF_CW * NS * 8 + (size_t)GF_CW * 32 * (p->naggs + 1) * 8 +
@@ -3543,12 +3876,21 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         bool done = false;
         vd_status st = try_q1(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
+        if (late_policy() == 2) {
+            st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done, true);
+            if (st != VD_OK || done) return st;
+        }
         st = try_scalar(p, cols, ncols, n, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_fkg(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_fkjs(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
+        if (late_policy() == 1) {
+            // branching scalar FK joins (Q19 shape): late loads beat the dense star fragment
+            st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done, true);
+            if (st != VD_OK || done) return st;
+        }
         st = try_star(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done);

@@ -1,9 +1,4 @@
-# Q9 FK grouped-fold iteration: parity of every variant + bench with L2 prefetch distances.
 set -x
 mkdir -p gpurun_out
-timeout 900 python -m pytest tests/test_gpu_pipeline.py -m gpu -q -p no:cacheprovider -k "q9" > gpurun_out/pytest_q9.log 2>&1; echo "pytest rc=$?" >> gpurun_out/pytest_q9.log
-timeout 900 python -m pytest tests/test_gpu_ops.py -m gpu -q -p no:cacheprovider -k "layout" > gpurun_out/pytest_layout.log 2>&1; echo "pytest rc=$?" >> gpurun_out/pytest_layout.log
-for pf in 0 2 4 8; do VD_FKP_PF=$pf timeout 300 python bench.py --workload q9 --no-cpu-baseline --no-e2e --steps 50 > gpurun_out/bench_q9_pf$pf.json 2>> gpurun_out/bench_q9.err; done
-VD_FKG_VARIANT=atom timeout 300 python bench.py --workload q9 --no-cpu-baseline --no-e2e --steps 50 > gpurun_out/bench_q9_atom.json 2>> gpurun_out/bench_q9.err
-timeout 600 ncu --set full --clock-control none --import-source on -k regex:k_pipe_fkg -s 1 -c 1 -o gpurun_out/prof_q9p -f python bench.py --workload q9 --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/ncu_q9p.log 2>&1
-timeout 1200 python -m pytest tests/test_gpu_fullsize.py -m gpu -q -p no:cacheprovider -k "q9" > gpurun_out/pytest_q9full.log 2>&1; echo "pytest rc=$?" >> gpurun_out/pytest_q9full.log
+for st in 4 3 2; do VD_FKG_STAGES=$st timeout 300 python bench.py --workload q9 --no-cpu-baseline --no-e2e --steps 100 > gpurun_out/bench_q9_st$st.json 2>> gpurun_out/bench_misc.err; done
+VD_FKG_STAGES=2 timeout 600 ncu --set full --clock-control none -k regex:k_pipe_fkg -s 1 -c 1 -o gpurun_out/prof_q9_st2 -f python bench.py --workload q9 --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/ncu_q9.log 2>&1

@@ -5,7 +5,9 @@
 //      per CTA), ld.shared::cluster.u8 through mapa
 //   2: local shared memory only (128 KiB per CTA, the upper bound)
 //   3: half of the lookups through DSMEM, half through L2
-// Prints lookups per ns for the whole GPU.
+// and the L2 slice throughput on B200 (k_l2): random 4-byte loads (one
+// sector each) and sequential 16-byte loads over a 64 MiB L2-resident buffer.
+// Prints lookups (sectors) per ns for the whole GPU.
 // nvcc -gencode arch=compute_100a,code=sm_100a -O3 -o scripts/ubench_gather scripts/ubench_gather.cu
 #include <cstdio>
 #include <cstdint>
@@ -67,6 +69,34 @@ __global__ void __cluster_dims__(8, 1, 1) __launch_bounds__(THREADS, 1)
     if (acc == 0xFFFFFFFFu) sink[0] = acc;
 }
 
+template <int SEQ>
+__global__ void __launch_bounds__(512) k_l2(const uint32_t* __restrict__ buf, uint32_t nwords, uint32_t* sink) {
+    uint32_t acc = 0;
+    const uint32_t tid = blockIdx.x * 512 + threadIdx.x;
+    if (SEQ) {
+        const uint4* b4 = reinterpret_cast<const uint4*>(buf);
+        const uint32_t nv = nwords / 4, stride = gridDim.x * 512;
+        for (int rep = 0; rep < 4; ++rep)
+            for (uint32_t i = tid; i < nv; i += stride * UNR) {
+                uint4 v[UNR];
+#pragma unroll
+                for (int u = 0; u < UNR; ++u) v[u] = i + u * stride < nv ? __ldcg(b4 + i + u * stride) : make_uint4(0, 0, 0, 0);
+#pragma unroll
+                for (int u = 0; u < UNR; ++u) acc += v[u].x ^ v[u].w;
+            }
+    } else {
+        uint32_t seed = tid * 0x9E3779B9u;
+        for (int it = 0; it < ITERS; it += UNR) {
+            uint32_t v[UNR];
+#pragma unroll
+            for (int u = 0; u < UNR; ++u) v[u] = __ldcg(buf + (hsh(seed + it + u) & (nwords - 1)));
+#pragma unroll
+            for (int u = 0; u < UNR; ++u) acc += v[u];
+        }
+    }
+    if (acc == 0xFFFFFFFFu) sink[0] = acc;
+}
+
 int main() {
     uint8_t* tbl;
     uint32_t* sink;
@@ -99,5 +129,29 @@ int main() {
     run(k_gather<1>, "dsmem_cluster8");
     run(k_gather<2>, "local_smem");
     run(k_gather<3>, "half_dsmem_half_l2");
+    {
+        const uint32_t nwords = 16u << 20;  // 64 MiB
+        uint32_t* buf;
+        cudaMalloc(&buf, (size_t)nwords * 4);
+        cudaMemset(buf, 3, (size_t)nwords * 4);
+        const int g = sms * 4;
+        for (int mode = 0; mode < 2; ++mode) {
+            auto kern = mode ? k_l2<1> : k_l2<0>;
+            for (int w = 0; w < 3; ++w) kern<<<g, 512>>>(buf, nwords, sink);
+            cudaEvent_t a, b;
+            cudaEventCreate(&a);
+            cudaEventCreate(&b);
+            cudaEventRecord(a);
+            for (int r = 0; r < 10; ++r) kern<<<g, 512>>>(buf, nwords, sink);
+            cudaEventRecord(b);
+            cudaEventSynchronize(b);
+            float ms = 0;
+            cudaEventElapsedTime(&ms, a, b);
+            const double sectors = mode ? 4.0 * nwords * 4 / 32 * 10 : (double)g * 512 * ITERS * 10;
+            printf("{\"route\": \"%s\", \"sectors_per_ns\": %.1f, \"GBps\": %.1f, \"err\": \"%s\"}\n",
+                   mode ? "l2_seq_ldg128" : "l2_random_sector", sectors / (ms * 1e6), sectors * 32 / (ms * 1e6),
+                   cudaGetErrorString(cudaGetLastError()));
+        }
+    }
     return 0;
 }

@@ -5,6 +5,9 @@ fragment (force_generic), in branching and predicated mode, on generated
 TPC-H-shaped tables that span many tiles with a ragged tail; integer /
 decimal aggregates bit-exact, the f64 selective sum within 1e-9 relative.
 """
+import contextlib
+import os
+
 import numpy as np
 import pytest
 import torch
@@ -36,6 +39,21 @@ def run(plan, views, n, dims=(), want=None):
     if want is not None:
         assert frag in want, (frag, want)
     return out.cpu().numpy().tobytes(), launches
+
+
+@contextlib.contextmanager
+def env(**kv):
+    """Set dispatch environment variables for the duration of a block."""
+    old = {k: os.environ.get(k) for k in kv}
+    os.environ.update(kv)
+    try:
+        yield
+    finally:
+        for k, v in old.items():
+            if v is None:
+                os.environ.pop(k, None)
+            else:
+                os.environ[k] = v
 
 
 def lineitem(sf, n=None, seed=gen.DEFAULT_SEED):
@@ -107,6 +125,9 @@ def test_q6_vs_oracle(sel_mode, generic, n):
     else:
         assert got == {0: [rev, cnt, cnt]}
     assert nl == 1
+    if sel_mode == vd.VD_SEL_BRANCH and not generic:
+        with env(VD_LATE="force"):  # late loads: l_shipdate leads, the rest per qualifying row
+            assert vd.decode_partials(run(plan, views, n, want=("late",))[0], plan) == got
 
 
 @pytest.mark.parametrize("sel_mode", [vd.VD_SEL_BRANCH, vd.VD_SEL_PREDICATED])
@@ -150,9 +171,13 @@ def test_fkj_q19_vs_oracle(sel_mode, generic, n):
     keep, views = load([li[c] for c in plans.Q19_COLS])
     dkeep, dviews = load([part[c] for c in plans.Q19_DIMS])
     plan = plans.q19(codes(), sel_mode, force_generic=generic)
-    got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews,
-                                 want=("generic",) if generic else ("star_join",))[0], plan)
+    frag = ("generic",) if generic else (("late",) if sel_mode == vd.VD_SEL_BRANCH else ("star_join",))
+    got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews, want=frag)[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+    if sel_mode == vd.VD_SEL_BRANCH and not generic:
+        with env(VD_LATE="off"):  # the dense star-join fragment on the same plan
+            got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews, want=("star_join",))[0], plan)
+        assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
 def test_fkj_q19_gather_fold_fragment():
@@ -164,12 +189,9 @@ def test_fkj_q19_gather_fold_fragment():
     exp = oracle.fkj(0, li, part, supp)
     keep, views = load([li[c] for c in plans.Q19_COLS])
     dkeep, dviews = load([part[c] for c in plans.Q19_DIMS])
-    os.environ["VD_STAR_VARIANT"] = "off"
-    try:
+    with env(VD_STAR_VARIANT="off", VD_LATE="off"):
         got = vd.decode_partials(run(plans.q19(codes()), views, len(li["l_partkey"]), dviews,
                                      want=("gather_fold",))[0], plans.q19(codes()))
-    finally:
-        del os.environ["VD_STAR_VARIANT"]
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
 
 
@@ -283,11 +305,17 @@ def test_star_join_random_predicates_vs_oracle(seed):
     dkeep, dviews = load([d1, d2, dr])
     plan = vd.pipeline(pred_=vd.pred(vconj), gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)],
                        aggs=[("sum", [2, (3, 100, -1)]), ("count",)])
-    got = vd.decode_partials(run(plan, views, n, dviews, want=("star_join",))[0], plan)
+    with env(VD_LATE="off"):
+        got = vd.decode_partials(run(plan, views, n, dviews, want=("star_join",))[0], plan)
     if exp_c == 0:
         assert got == {}
     else:
         assert got == {0: [int(exp_s), int(exp_c), int(exp_c)]}
+    # default dispatch (the late-materialisation fragment when the conjunctions
+    # share interval terms on u8 / i32 columns) and the general gather-fold one
+    assert vd.decode_partials(run(plan, views, n, dviews, want=("star_join", "late"))[0], plan) == got
+    with env(VD_LATE="off", VD_STAR_VARIANT="off"):
+        assert vd.decode_partials(run(plan, views, n, dviews, want=("gather_fold",))[0], plan) == got
     gen_plan = vd.pipeline(pred_=vd.pred(vconj), gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)],
                            aggs=[("sum", [2, (3, 100, -1)]), ("count",)], force_generic=True)
     assert vd.decode_partials(run(gen_plan, views, n, dviews, want=("generic",))[0], gen_plan) == got
@@ -516,3 +544,70 @@ def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel, variant):
         assert got == {}
     else:
         assert got == {0: [exp_s or 0, exp_c, exp_c]}
+
+
+@pytest.mark.parametrize("seed", range(10))
+def test_late_fragment_random_plans_vs_oracle(seed):
+    """Late-materialisation fragment on random branching plans: terms shared
+    by every conjunction on two u8 columns and one i32 column (the lead
+    columns: intervals, IN sets and NE that are not, epsilon in every column),
+    per-conjunction terms on the other columns, a ragged row count; against
+    the oracle (one FoldSelect program per conjunction, union, then Gather ->
+    Multiply -> FoldSum / FoldCount)."""
+    rng = np.random.default_rng(700 + seed)
+    n = 50001 + 37 * seed  # n % 16 != 0: the tail rows
+    cols = {"a": rng.integers(0, 40, n).astype(np.uint8), "b": rng.integers(0, 8, n).astype(np.uint8),
+            "c": rng.integers(-500, 500, n).astype(np.int32), "x": rng.integers(0, 10**6, n).astype(np.int64),
+            "y": rng.integers(0, 11, n).astype(np.int64), "r": rng.integers(0, 100, n).astype(np.int64)}
+    eps = {}
+    for k, arr in cols.items():
+        m = rng.random(n) < 0.01
+        arr[m] = {np.uint8: 255, np.int32: -2**31, np.int64: -2**63}[arr.dtype.type]
+        eps[k] = m
+    order = ["a", "b", "c", "x", "y", "r"]
+    idx = {k: i for i, k in enumerate(order)}
+
+    def term(k):
+        if k in ("a", "b"):
+            cmp = str(rng.choice([">", "<", ">=", "<=", "==", "!=", "in"]))
+            if cmp == "in":
+                lo = int(rng.integers(0, 30))
+                return k, cmp, (list(range(lo, lo + int(rng.integers(1, 6)))) if rng.random() < 0.6
+                                else sorted(set(int(v) for v in rng.integers(0, 40, 4))))
+            return k, cmp, int(rng.integers(0, 40 if k == "a" else 8))
+        if k == "c":
+            return k, str(rng.choice([">", "<", ">=", "<=", "=="], p=[.3, .3, .15, .15, .1])), int(rng.integers(-400, 400))
+        return k, str(rng.choice([">", "<", ">=", "<="])), int(rng.integers(0, 100))
+
+    common = [term(k) for k in ("a", "b") if rng.random() < 0.8] + [term("c")]  # c: always an interval lead
+    conjs = [common + [term("r") for _ in range(int(rng.integers(0, 3)))] for _ in range(int(rng.integers(1, 4)))]
+    sel = np.zeros(n, dtype=bool)
+    inputs = {f"fact__{k}": (v, eps[k]) for k, v in cols.items()}
+    for terms in conjs:
+        lines, names = [], []
+        for j, (k, cmp, val) in enumerate(terms):
+            _term_expr(f"t{j}", f"fact.{k}", cmp, val, lines)
+            names.append(f"t{j}")
+        lines.append(f"q := LogicalAnd({names[0]}, {names[0]})")
+        for nm in names[1:]:
+            lines.append(f"q := LogicalAnd(q, {nm})")
+        lines.append("pos := FoldSelect(q)")
+        pos, pe = oracle.run("\n".join(lines), **inputs).get_arrays("pos")
+        sel[pos[~pe]] = True
+    upos = np.nonzero(sel)[0].astype(np.int64)
+    agg = oracle.run("""
+    gx := Gather(fact.x, pos)
+    gy := Gather(fact.y, pos)
+    f := Multiply(gy, -1)
+    t := Add(f, 100)
+    pr := Multiply(gx, t)
+    s := FoldSum(pr)
+    c := FoldCount(pos)
+    """, fact__x=(cols["x"], eps["x"]), fact__y=(cols["y"], eps["y"]), pos=upos)
+    exp = {0: [int(agg.get("s")[0]), int(agg.get("c")[0]), int(agg.get("c")[0])]} if upos.size else {}
+    keep, views = load([cols[k] for k in order])
+    plan = vd.pipeline(pred_=vd.pred([[(idx[k], cmp, val) for k, cmp, val in t] for t in conjs]),
+                       aggs=[("sum", [idx["x"], (idx["y"], 100, -1)]), ("count",)])
+    with env(VD_LATE="force"):
+        got = vd.decode_partials(run(plan, views, n, want=("late",))[0], plan)
+    assert got == exp
