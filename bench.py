@@ -367,6 +367,14 @@ def main():
         looked_up = n if args.sel_mode == "predicated" else sel_rows // max(world, 1)
         alg_bytes = n * bpr + 64 * looked_up
         extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64}
+    elif w == "q19" and vd.last_fragment() == "late":
+        # late-materialisation fragment, readings A31/A33: the lead columns
+        # (l_shipmode, l_shipinstruct: the u8 terms every conjunction shares)
+        # in full; of l_partkey / l_quantity the 64-byte blocks holding a
+        # lead-qualified row, of l_extendedprice / l_discount those holding a
+        # qualifying row; the part table (120 MB at SF100, L2-sized) once;
+        # the lookups themselves are L2 sectors (roofline.l2)
+        alg_bytes, extra = q19_late_bytes(plan, cols, dims, result, clk, kernel_ms)
     elif w in ("q9", "q19"):
         # the dimension lookups hit L2 (supplier 1 MB; part 120 MB at SF100):
         # the second bound is L2 slice throughput, one 32-byte sector per
@@ -400,7 +408,7 @@ def main():
                          "q9": f"fkj_q9_sf{sf:g}", "select": f"select_f32_{n_total}_s{args.selectivity:g}",
                          "fkjsel": f"fkjsel_{n_total}x{plans.FKJSEL_TARGET_ROWS}_s{args.selectivity:g}"}[w],
             "rows": n_total, "rows_per_gpu": n, "sf": sf, "sel_mode": args.sel_mode,
-            "fragment": "generic" if args.generic else "specialised",
+            "fragment": "generic" if args.generic else vd.last_fragment(),
             "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
             "l2": f"inputs {n * bpr / 1e9:.1f} GB per GPU > 126 MB L2: no flush needed",
             "seed": args.seed,
@@ -696,6 +704,63 @@ def fig14_main(args, rank, world, local):
     if rank == 0:
         print(json.dumps(line), flush=True)
     comm.close()
+
+
+def q19_late_bytes(plan, cols, dims, result, clk, kernel_ms):
+    """Algorithmic bytes of the Q19 late-materialisation fragment (A31/A33)."""
+    import torch
+
+    import gen
+    from paper_journals_pvldb_pirkmzm16_b200 import plans
+    mode, instr = cols[4], cols[5]
+    codes_m = [i for i, s in enumerate(gen.SHIPMODE) if s in ("AIR", "AIR REG")]
+    lead = (instr == gen.SHIPINSTRUCT.index("DELIVER IN PERSON"))
+    lead &= torch.isin(mode, torch.tensor(codes_m, dtype=mode.dtype, device=mode.device))
+    n = lead.numel()
+
+    def blocks(mask, esz):
+        r = 64 // esz
+        full = n // r * r
+        return 64 * (int(mask[:full].view(-1, r).any(1).sum().item()) + int(bool(mask[full:].any().item())))
+
+    nlead = int(lead.sum().item())
+    qual = int(next(iter(result.values()))[-1]) if result else 0
+    # k_pipe_late's order: l_partkey, then the equality / IN lookups (p_brand,
+    # p_container); l_quantity and p_size only for rows those leave undecided
+    # (some branch's brand and container match); the aggregate inputs only
+    # for qualifying rows
+    idx = lead.nonzero().squeeze(1)
+    pk = cols[0][idx].long() - 1
+    br, ct = dims[0][pk].long(), dims[1][pk].long()
+    und = torch.zeros_like(br, dtype=torch.bool)
+    for b, conts, _, _ in plans.Q19_BRANCHES:
+        und |= (br == gen.BRAND.index(b)) & torch.isin(ct, torch.tensor([gen.CONTAINER.index(x) for x in conts],
+                                                                         device=ct.device))
+    iu = idx[und]
+    qty, sz = cols[1][iu].long(), dims[2][pk[und]].long()
+    ok = torch.zeros_like(qty, dtype=torch.bool)
+    for b, conts, qlo, smax in plans.Q19_BRANCHES:
+        ok |= ((br[und] == gen.BRAND.index(b))
+               & torch.isin(ct[und], torch.tensor([gen.CONTAINER.index(x) for x in conts], device=ct.device))
+               & (qty >= qlo * 100) & (qty <= (qlo + 10) * 100) & (sz >= 1) & (sz <= smax))
+    und_mask = torch.zeros(n, dtype=torch.bool, device=lead.device)
+    und_mask[iu] = True
+    full_mask = torch.zeros(n, dtype=torch.bool, device=lead.device)
+    full_mask[iu[ok]] = True
+    alg = 2 * n + blocks(lead, cols[0].element_size()) + blocks(und_mask, cols[1].element_size())
+    alg += blocks(full_mask, cols[2].element_size()) + blocks(full_mask, cols[3].element_size())
+    alg += sum(d.numel() * d.element_size() for d in dims)
+    clk_ghz = (clk or {}).get("sm_mhz") or 1965.0
+    cap = L2_CAP_BYTES_PER_CLK * clk_ghz / 1e3 / 32
+    nund = int(und.sum().item())
+    sectors = 2 * nlead + nund
+    ach = sectors / (kernel_ms * 1e6)
+    extra = {"bytes_per_row_dense": BYTES_PER_ROW["q19"], "lead_rows": nlead, "undecided_rows": nund,
+             "qualifying_rows": qual, "qualifying_check": int(ok.sum().item()),
+             "l2": {"bound": "l2", "lookups": sectors, "achieved_lookups_only": ach, "peak": cap,
+                    "unit": "sectors/ns", "frac": ach / cap,
+                    "peak_kind": "guide: B300-measured LTS cap 6300 B/clk x SM clock (B300_MICROARCH.md)"}}
+    return alg, extra
 
 
 def q15_main(args, rank, world, local, sf):

@@ -1363,6 +1363,11 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
 // A dense TMA fragment moves every byte of every column; this one moves the
 // lead bytes plus the 64-byte blocks that hold a qualifying row.
 // ============================================================================
+struct LtCons {
+    int32_t ref, pad;
+    int64_t lo, hi;
+    uint64_t in;
+};
 struct LateLead {
     const uint8_t* c8[2];
     uint32_t lo8[2], hi8[2];  // interval bounds replicated into the 4 bytes
@@ -1370,49 +1375,156 @@ struct LateLead {
     int32_t lo32, hi32;       // lo32 > INT32_MIN: epsilon never passes
     // references (bit c: base column c, bit ncols + g: gather g) read by the
     // rest of the predicate / by the aggregates; FK columns of the gathers
-    // included, so that each group of loads is issued at once
-    uint32_t pref, aref;
+    // included, so that each group of loads is issued at once.  pref1 (a
+    // subset of pref): the references of the equality / IN terms, loaded
+    // first; the rest of pref only for rows those terms leave undecided
+    uint32_t pref, pref1, aref;
+    // the predicate compiled to one constraint per (conjunction, reference):
+    // lo <= x <= hi and bit x of `in` (IN sets; ~0 = none), epsilon fails.
+    // Row VD_MAX_CONJ holds the common terms.  ncons[0] < 0: a term (NE)
+    // has no such form and the term lists of GfArgs are interpreted instead
+    int32_t ncons[VD_MAX_CONJ + 1];
+    LtCons cons[VD_MAX_CONJ + 1][VD_MAX_TERMS];
 };
 
-// A lead-qualified row: the predicate's columns and lookups are loaded in
-// two rounds (base columns, then the dimension lookups they address), all
-// loads of a round in flight together; the aggregate inputs are loaded only
-// when the row qualifies (late materialisation).
-__device__ __forceinline__ void late_load(const GfArgs& a, uint32_t want, uint32_t have, int64_t row, Val* v) {
-#pragma unroll
-    for (int c = 0; c < GF_MAXCOLS; ++c)
-        if (c < a.ncols && ((want & ~have) >> c & 1u)) v[c] = fetch_typed(a.col[c], a.dt[c], row);
-#pragma unroll
-    for (int g = 0; g < VD_MAX_GATHERS; ++g) {
-        const int r = a.ncols + g;
-        if (g < a.ngathers && ((want & ~have) >> r & 1u)) {
-            const Val fk = v[a.g_fk[g]];
-            const int64_t p = fk.i - a.g_bias[g];
-            if (fk.eps || p < 0 || p >= a.g_len[g]) {
-                v[r].eps = true;
-                v[r].isf = false;
-                v[r].i = 0;
-                v[r].f = 0;
-            } else {
-                v[r] = fetch_typed(a.g_p[g], a.g_dt[g], p);
-            }
-        }
-    }
+// L2 eviction policy for data re-read by other rows (the dimension lookups).
+__device__ __forceinline__ uint64_t policy_evict_last() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
 }
 
-__device__ __forceinline__ bool late_pred(const GfArgs& a, const Val* v) {
-    for (int k = 0; k < a.ncommon; ++k)
-        if (!term_true(a.common[k], v[a.common[k].col])) return false;
-    if (a.pred.nconj == 0) return true;
-    for (int c = 0; c < a.pred.nconj; ++c) {
-        bool ok = true;
-        for (int k = 0; k < a.pred.nterms[c] && ok; ++k) ok = term_true(a.pred.t[c][k], v[a.pred.t[c][k].col]);
-        if (ok) return true;
-    }
-    return false;
-}
 constexpr int LT_THREADS = 256;
 constexpr int LT_QCAP = 32 + 16 * 32;  // < 32 left over + one 16-row step of every lane
+// dynamic shared memory of the largest plan (values, accumulators, queues)
+constexpr int LT_SMEM_MAX = (GF_MAXCOLS + VD_MAX_GATHERS + VD_MAX_AGGS + 1) * LT_THREADS * 8 + (LT_THREADS / 32) * LT_QCAP * 4;
+
+// Late loads of one row go straight to shared memory (cp.async, no
+// registers held while in flight): every referenced base column at once,
+// then the lookups they address.  The thread's values live in its column of
+// sv[ref][LT_THREADS] (dynamic reference indices stay in shared memory, not
+// in spilled local memory), widened to int64 with epsilon = INT64_MIN.  A u8
+// element travels in its aligned 4-byte word (cp.async moves 4, 8 or 16
+// bytes), unless that word would run past the column's end.
+__device__ __forceinline__ void lt_cp(int64_t* sdst, const void* col, int32_t dt, int64_t i, int64_t len,
+                                      uint64_t pol) {
+    if (dt == VD_I64) {
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 8, %2;" ::"r"(smem_u32(sdst)),
+                     "l"((const int64_t*)col + i), "l"(pol)
+                     : "memory");
+    } else if (dt == VD_I32) {
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
+                     "l"((const int32_t*)col + i), "l"(pol)
+                     : "memory");
+    } else if ((i | 3) < len) {
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
+                     "l"((const uint8_t*)col + (i & ~(int64_t)3)), "l"(pol)
+                     : "memory");
+    } else {
+        *reinterpret_cast<uint32_t*>(sdst) = (uint32_t)__ldg((const uint8_t*)col + i) << (8 * (i & 3));
+    }
+}
+__device__ __forceinline__ int64_t lt_decode(const int64_t* sv, int32_t dt, int64_t i) {
+    if (dt == VD_I64) return *sv;
+    const uint32_t w = *reinterpret_cast<const uint32_t*>(sv);
+    if (dt == VD_I32) return (int32_t)w == INT32_MIN ? INT64_MIN : (int64_t)(int32_t)w;
+    const uint32_t x = (w >> (8 * (i & 3))) & 0xFFu;
+    return x == 0xFFu ? INT64_MIN : (int64_t)x;
+}
+__device__ __forceinline__ void cp_async_wait_all() {
+    asm volatile("cp.async.commit_group;\n\tcp.async.wait_group 0;" ::: "memory");
+}
+
+__device__ __forceinline__ void late_load(const GfArgs& a, uint32_t want, int64_t row, int64_t (*sv)[LT_THREADS],
+                                          int tid, uint64_t pol_s, uint64_t pol_d) {
+    const uint32_t wb = want & ((1u << a.ncols) - 1);
+    for (uint32_t m = wb; m; m &= m - 1) {
+        const int c = __ffs(m) - 1;
+        lt_cp(&sv[c][tid], a.col[c], a.dt[c], row, a.n, pol_s);
+    }
+    cp_async_wait_all();
+    for (uint32_t m = wb; m; m &= m - 1) {
+        const int c = __ffs(m) - 1;
+        sv[c][tid] = lt_decode(&sv[c][tid], a.dt[c], row);
+    }
+    const uint32_t wg = want >> a.ncols;
+    if (!wg) return;
+    int64_t pidx[VD_MAX_GATHERS];
+#pragma unroll
+    for (int g = 0; g < VD_MAX_GATHERS; ++g) {
+        if (!((wg >> g) & 1u)) continue;
+        const int64_t fk = sv[a.g_fk[g]][tid];
+        pidx[g] = fk - a.g_bias[g];
+        if (fk == INT64_MIN || pidx[g] < 0 || pidx[g] >= a.g_len[g]) {
+            pidx[g] = -1;
+            sv[a.ncols + g][tid] = INT64_MIN;
+        } else {
+            lt_cp(&sv[a.ncols + g][tid], a.g_p[g], a.g_dt[g], pidx[g], a.g_len[g], pol_d);
+        }
+    }
+    cp_async_wait_all();
+#pragma unroll
+    for (int g = 0; g < VD_MAX_GATHERS; ++g)
+        if (((wg >> g) & 1u) && pidx[g] >= 0) sv[a.ncols + g][tid] = lt_decode(&sv[a.ncols + g][tid], a.g_dt[g], pidx[g]);
+}
+
+// Three-valued predicate over the references loaded so far (`known`): a term
+// on a reference not yet loaded is unknown.  Returns 0 (false), 1 (true) or
+// 2 (undecided: load the rest and evaluate again).
+__device__ __forceinline__ int late_term(const DevTerm& t, const int64_t (*sv)[LT_THREADS], int tid, uint32_t known) {
+    if (!((known >> t.col) & 1u)) return 2;
+    const int64_t x = sv[t.col][tid];
+    return x != INT64_MIN && cmp_int(t.cmp, x, t.iv);  // epsilon is "not selected" (A9)
+}
+
+__device__ __forceinline__ int late_pred(const GfArgs& a, const int64_t (*sv)[LT_THREADS], int tid, uint32_t known) {
+    int r = 1;
+    for (int k = 0; k < a.ncommon; ++k) {
+        const int t = late_term(a.common[k], sv, tid, known);
+        if (t == 0) return 0;
+        r = t == 2 ? 2 : r;
+    }
+    if (a.pred.nconj == 0) return r;
+    int any = 0;  // 0: every conjunction false so far, 2: one undecided
+    for (int c = 0; c < a.pred.nconj; ++c) {
+        int cj = 1;
+        for (int k = 0; k < a.pred.nterms[c] && cj != 0; ++k) {
+            const int t = late_term(a.pred.t[c][k], sv, tid, known);
+            cj = t == 0 ? 0 : (t == 2 ? 2 : cj);
+        }
+        if (cj == 1) return r;  // true, unless a common term is undecided
+        if (cj == 2) any = 2;
+    }
+    return any;
+}
+
+// The same over the compiled constraints (no per-term comparison switch).
+__device__ __forceinline__ int late_cons(const LtCons* cs, int n, const int64_t (*sv)[LT_THREADS], int tid,
+                                         uint32_t known) {
+    int r = 1;
+    for (int k = 0; k < n; ++k) {
+        const LtCons& c = cs[k];
+        if (!((known >> c.ref) & 1u)) {
+            r = 2;
+            continue;
+        }
+        const int64_t x = sv[c.ref][tid];
+        if (x == INT64_MIN || x < c.lo || x > c.hi || !((c.in >> (x & 63)) & 1ull)) return 0;
+    }
+    return r;
+}
+__device__ __forceinline__ int late_pred_c(const LateLead& ld, int nconj, const int64_t (*sv)[LT_THREADS], int tid,
+                                           uint32_t known) {
+    const int r = late_cons(ld.cons[VD_MAX_CONJ], ld.ncons[VD_MAX_CONJ], sv, tid, known);
+    if (r == 0 || nconj == 0) return r;
+    int any = 0;
+    for (int c = 0; c < nconj; ++c) {
+        const int cj = late_cons(ld.cons[c], ld.ncons[c], sv, tid, known);
+        if (cj == 1) return r;
+        if (cj == 2) any = 2;
+    }
+    return any;
+}
 
 // 16 u8 rows (one 128-bit word) against [lo, hi] per byte -> 16-bit mask
 __device__ __forceinline__ uint32_t lt_mask_u8(int4 v, uint32_t lo4, uint32_t hi4) {
@@ -1425,31 +1537,55 @@ __device__ __forceinline__ uint32_t lt_mask_u8(int4 v, uint32_t lo4, uint32_t hi
     }
     return m;
 }
+__device__ __forceinline__ uint32_t lt_mask_i32(const int4 (&v)[4], int32_t lo, int32_t hi) {
+    uint32_t m = 0;
+#pragma unroll
+    for (int k = 0; k < 4; ++k) {
+        const int32_t x[4] = {v[k].x, v[k].y, v[k].z, v[k].w};
+#pragma unroll
+        for (int j = 0; j < 4; ++j) m |= (uint32_t)(x[j] >= lo && x[j] <= hi) << (4 * k + j);
+    }
+    return m;
+}
+__device__ __forceinline__ int4 lt_ld16(const void* p, uint64_t pol) {
+    int4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.L2::cache_hint.v4.s32 {%0,%1,%2,%3}, [%4], %5;"
+                 : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w)
+                 : "l"(p), "l"(pol));
+    return r;
+}
 
 template <int N8, bool I32>
-__global__ void __launch_bounds__(LT_THREADS) k_pipe_late(const __grid_constant__ GfArgs a,
+__global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_constant__ GfArgs a,
                                                          const __grid_constant__ LateLead ld,
                                                          Slot16* __restrict__ parts, unsigned int* __restrict__ done,
                                                          Slot16* __restrict__ out) {
-    __shared__ int32_t s_q[LT_THREADS / 32][LT_QCAP];
+    // dynamic shared memory: per-thread values [ref][thread], per-thread
+    // accumulators [agg][thread] (touched by qualifying rows only, kept out
+    // of the register file), per-warp row queues
+    extern __shared__ __align__(16) uint8_t lt_smem[];
+    // (sized by the plan: ncols + ngathers value rows, naggs + 1 accumulator rows)
+    const int NA = a.naggs, nref = a.ncols + a.ngathers;
+    int64_t(*s_v)[LT_THREADS] = reinterpret_cast<int64_t(*)[LT_THREADS]>(lt_smem);
+    int64_t(*s_a)[LT_THREADS] = reinterpret_cast<int64_t(*)[LT_THREADS]>(lt_smem + nref * LT_THREADS * 8);
+    int32_t(*s_q)[LT_QCAP] = reinterpret_cast<int32_t(*)[LT_QCAP]>(lt_smem + (nref + NA + 1) * LT_THREADS * 8);
     __shared__ int64_t s_acc[LT_THREADS / 32][VD_MAX_AGGS + 1];
-    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int NA = a.naggs;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, tid = threadIdx.x;
+    const uint64_t pol_s = policy_evict_first(), pol_d = policy_evict_last();
     int32_t* q_ = s_q[warp];
     int cnt = 0;  // warp-uniform queue depth
-    int64_t racc[VD_MAX_AGGS + 1];
-#pragma unroll
-    for (int g = 0; g <= VD_MAX_AGGS; ++g) racc[g] = 0;
+    for (int g = 0; g <= NA; ++g) s_a[g][tid] = 0;
     // the rest of the predicate and the aggregate inputs of one lead-qualified row
     auto fold_row = [&](int64_t row) {
-        Val v[GF_MAXCOLS + VD_MAX_GATHERS];
-        const uint32_t pb = ld.pref & ((1u << a.ncols) - 1);
-        late_load(a, pb, 0, row, v);               // round 1: base columns of the predicate (+ FKs)
-        late_load(a, ld.pref & ~pb, pb, row, v);   // round 2: the lookups they address
-        if (!late_pred(a, v)) return;
-        const uint32_t ab = ld.aref & ((1u << a.ncols) - 1);
-        late_load(a, ab, ld.pref, row, v);
-        late_load(a, ld.aref & ~ab, ld.pref | ab, row, v);
+        late_load(a, ld.pref1, row, s_v, tid, pol_s, pol_d);
+        const bool compiled = ld.ncons[0] >= 0;
+        int t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1) : late_pred(a, s_v, tid, ld.pref1);
+        if (t == 2) {
+            late_load(a, ld.pref & ~ld.pref1, row, s_v, tid, pol_s, pol_d);
+            t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref) : late_pred(a, s_v, tid, ld.pref);
+        }
+        if (t != 1) return;
+        late_load(a, ld.aref & ~ld.pref, row, s_v, tid, pol_s, pol_d);
 #pragma unroll
         for (int g = 0; g < VD_MAX_AGGS; ++g) {
             if (g >= NA) break;
@@ -1459,17 +1595,16 @@ __global__ void __launch_bounds__(LT_THREADS) k_pipe_late(const __grid_constant_
                 for (int f = 0; f < a.a_nf[g]; ++f) {
                     int64_t x = 0;
                     if (a.a_col[g][f] >= 0) {
-                        const Val& u = v[a.a_col[g][f]];
-                        e |= u.eps;
-                        x = u.i;
+                        x = s_v[a.a_col[g][f]][tid];
+                        e |= x == INT64_MIN;
                     }
                     pr *= a.a_a[g][f] + a.a_b[g][f] * x;
                 }
                 if (e) pr = 0;  // an epsilon input is skipped by the fold (A5)
             }
-            racc[g] += pr;
+            s_a[g][tid] += pr;
         }
-        racc[VD_MAX_AGGS] += 1;
+        s_a[NA][tid] += 1;
     };
     auto drain = [&](int k) {  // fold the top k (<= 32) queued rows
         __syncwarp();
@@ -1479,24 +1614,30 @@ __global__ void __launch_bounds__(LT_THREADS) k_pipe_late(const __grid_constant_
     };
     const int64_t nq = a.n / 16;
     const int64_t wstride = (int64_t)gridDim.x * LT_THREADS;
-    for (int64_t q0 = (int64_t)blockIdx.x * LT_THREADS + warp * 32; q0 < nq; q0 += wstride) {
+    // lead words of the current step, and of the next one loaded before the
+    // current step's drain (the stream stays in flight behind the late loads)
+    int4 c8[N8 > 0 ? N8 : 1], c32[4];
+    auto load_lead = [&](int64_t q, int4* w8, int4* w32) {
+        if (q >= nq) return;
+#pragma unroll
+        for (int j = 0; j < N8; ++j) w8[j] = lt_ld16(ld.c8[j] + 16 * q, pol_s);
+        if (I32) {
+#pragma unroll
+            for (int k = 0; k < 4; ++k) w32[k] = lt_ld16(ld.c32 + 16 * q + 4 * k, pol_s);
+        }
+    };
+    int64_t q0 = (int64_t)blockIdx.x * LT_THREADS + warp * 32;
+    load_lead(q0 + lane, c8, c32);
+    for (; q0 < nq; q0 += wstride) {
         const int64_t q = q0 + lane;
         uint32_t m = 0;
         if (q < nq) {
             m = 0xFFFFu;
 #pragma unroll
-            for (int j = 0; j < N8; ++j) m &= lt_mask_u8(ld_stream16(ld.c8[j] + 16 * q), ld.lo8[j], ld.hi8[j]);
-            if (I32) {
-#pragma unroll
-                for (int k = 0; k < 4; ++k) {
-                    const int4 v = ld_stream16(ld.c32 + 16 * q + 4 * k);
-                    const int32_t x[4] = {v.x, v.y, v.z, v.w};
-#pragma unroll
-                    for (int j = 0; j < 4; ++j)
-                        if (x[j] < ld.lo32 || x[j] > ld.hi32) m &= ~(1u << (4 * k + j));
-                }
-            }
+            for (int j = 0; j < N8; ++j) m &= lt_mask_u8(c8[j], ld.lo8[j], ld.hi8[j]);
+            if (I32) m &= lt_mask_i32(c32, ld.lo32, ld.hi32);
         }
+        load_lead(q + wstride, c8, c32);
         // compaction: the lanes' qualifying rows, in row order, onto the warp's queue
         const int pc = __popc(m);
         int incl = pc;
@@ -1529,15 +1670,14 @@ __global__ void __launch_bounds__(LT_THREADS) k_pipe_late(const __grid_constant_
         }
     }
     // fold: warp sums (int64, bounded on the host) -> CTA (int128) -> last CTA
-#pragma unroll
-    for (int g = 0; g <= VD_MAX_AGGS; ++g) {
-        const int64_t t = warp_sum_i64(racc[g]);
+    for (int g = 0; g <= NA; ++g) {
+        const int64_t t = warp_sum_i64(s_a[g][tid]);
         if (lane == 0) s_acc[warp][g] = t;
     }
     __syncthreads();
     const int NS = NA + 1;
     if (threadIdx.x < NS) {
-        const int g = threadIdx.x < NA ? threadIdx.x : VD_MAX_AGGS;
+        const int g = threadIdx.x;  // aggregates, then the row count
         i128 t = 0;
         for (int w = 0; w < LT_THREADS / 32; ++w) t += (i128)s_acc[w][g];
         put_i128(&parts[(size_t)blockIdx.x * NS + threadIdx.x], t);
@@ -3709,19 +3849,82 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
             m |= 1u << c;
             if (c >= ncols) m |= 1u << A.g_fk[c - ncols];
         };
-        for (int k = 0; k < A.ncommon; ++k) ref(L.pref, A.common[k].col);
+        auto selective = [](int cmp) { return cmp == VD_CMP_EQ || cmp == VD_CMP_IN; };
+        for (int k = 0; k < A.ncommon; ++k) {
+            ref(L.pref, A.common[k].col);
+            if (selective(A.common[k].cmp)) ref(L.pref1, A.common[k].col);
+        }
         for (int c = 0; c < A.pred.nconj; ++c)
-            for (int k = 0; k < A.pred.nterms[c]; ++k) ref(L.pref, A.pred.t[c][k].col);
+            for (int k = 0; k < A.pred.nterms[c]; ++k) {
+                ref(L.pref, A.pred.t[c][k].col);
+                if (selective(A.pred.t[c][k].cmp)) ref(L.pref1, A.pred.t[c][k].col);
+            }
+        // no equality / IN term: one round over every predicate reference
+        if (L.pref1 == 0) L.pref1 = L.pref;
+        // compile the terms into per-reference constraints (IN: 0 <= x < 64)
+        auto compile = [&](const DevTerm* ts, int nt, LtCons* out) -> int {
+            int nc = 0;
+            for (int k = 0; k < nt; ++k) {
+                const DevTerm& t = ts[k];
+                int at = -1;
+                for (int h = 0; h < nc; ++h) at = out[h].ref == t.col ? h : at;
+                if (at < 0) {
+                    at = nc++;
+                    out[at].ref = t.col;
+                    out[at].pad = 0;
+                    out[at].lo = INT64_MIN + 1;
+                    out[at].hi = INT64_MAX;
+                    out[at].in = ~0ull;
+                }
+                LtCons& c = out[at];
+                const int64_t v = t.iv;
+                switch (t.cmp) {
+                case VD_CMP_GT: if (v == INT64_MAX) c.hi = c.lo - 1; else c.lo = std::max(c.lo, v + 1); break;
+                case VD_CMP_GE: c.lo = std::max(c.lo, v); break;
+                case VD_CMP_LT: if (v == INT64_MIN) c.hi = c.lo - 1; else c.hi = std::min(c.hi, v - 1); break;
+                case VD_CMP_LE: c.hi = std::min(c.hi, v); break;
+                case VD_CMP_EQ: c.lo = std::max(c.lo, v); c.hi = std::min(c.hi, v); break;
+                case VD_CMP_IN: c.in &= (uint64_t)v; c.lo = std::max(c.lo, (int64_t)0); c.hi = std::min(c.hi, (int64_t)63); break;
+                default: return -1;  // NE
+                }
+            }
+            return nc;
+        };
+        bool ok = true;
+        L.ncons[VD_MAX_CONJ] = compile(A.common, A.ncommon, L.cons[VD_MAX_CONJ]);
+        ok = L.ncons[VD_MAX_CONJ] >= 0;
+        for (int c = 0; c < A.pred.nconj && ok; ++c) {
+            L.ncons[c] = compile(A.pred.t[c], A.pred.nterms[c], L.cons[c]);
+            ok = L.ncons[c] >= 0;
+        }
+        if (!ok) L.ncons[0] = -1;
+        else if (A.pred.nconj == 0) L.ncons[0] = 0;
         for (int g = 0; g < A.naggs; ++g)
             if (A.a_kind[g] != VD_AGG_COUNT)
                 for (int f = 0; f < A.a_nf[g]; ++f)
                     if (A.a_col[g][f] >= 0) ref(L.aref, A.a_col[g][f]);
-        const int grid = grid_persistent(4);  // the pipeline workspace holds 4 x SMs partial slots
+        // the late loads are integer (epsilon = INT64_MIN after widening)
+        for (int c = 0; c < ncols; ++c)
+            if ((((L.pref | L.aref) >> c) & 1u) && !is_int(cols[c].dtype)) return VD_OK;
+        // one wave: as many CTAs per SM as fit (registers allow 4; the
+        // pipeline workspace holds 4 x SMs partial slots)
+        const size_t lsm = (size_t)(ncols + p->ngathers + p->naggs + 1) * LT_THREADS * 8 +
+                           (size_t)(LT_THREADS / 32) * LT_QCAP * 4;
+        const int per_sm = std::max(1, std::min(4, (int)((220 * 1024) / (lsm + 1024))));
+        const int grid = grid_persistent(per_sm);
         unsigned int* dn = (unsigned int*)ws;
         Slot16* parts = (Slot16*)((char*)ws + 256);
         cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-#define LT_GO(N8_, I32_) k_pipe_late<N8_, I32_><<<grid, LT_THREADS, 0, s>>>(A, L, parts, dn, (Slot16*)out)
+#define LT_GO(N8_, I32_)                                                                                    \
+    do {                                                                                                    \
+        static bool attr_ = false;                                                                          \
+        if (!attr_) {                                                                                       \
+            cudaFuncSetAttribute(k_pipe_late<N8_, I32_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
+            attr_ = true;                                                                                   \
+        }                                                                                                   \
+        k_pipe_late<N8_, I32_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);               \
+    } while (0)
         if (n8 == 2) { if (i32) LT_GO(2, true); else LT_GO(2, false); }
         else if (n8 == 1) { if (i32) LT_GO(1, true); else LT_GO(1, false); }
         else LT_GO(0, true);

@@ -52,6 +52,13 @@ def selsum(t: float, sel_mode=VD_SEL_BRANCH, force_generic=False):
                     force_generic=force_generic)
 
 
+# the three branches of TPC-H Q19: brand, containers, quantity lower bound
+# (the upper is +10), maximum p_size
+Q19_BRANCHES = [("Brand#12", ["SM CASE", "SM BOX", "SM PACK", "SM PKG"], 1, 5),
+                ("Brand#23", ["MED BAG", "MED BOX", "MED PKG", "MED PACK"], 10, 10),
+                ("Brand#34", ["LG CASE", "LG BOX", "LG PACK", "LG PKG"], 20, 15)]
+
+
 def q19(codes, sel_mode=VD_SEL_BRANCH, force_generic=False):
     """Q19-style FK gather join (C5): lineitem x part through l_partkey - 1,
     the three-branch disjunctive predicate of TPC-H Q19, sum(ext*(100-disc)).
@@ -60,9 +67,7 @@ def q19(codes, sel_mode=VD_SEL_BRANCH, force_generic=False):
     B, C, M, I_ = codes["brand"], codes["container"], codes["shipmode"], codes["shipinstruct"]
     modes = [M[m] for m in ("AIR", "AIR REG") if m in M]  # 'AIR REG' is not a dbgen value (A26)
     conjs = []
-    for brand, conts, qlo, smax in [("Brand#12", ["SM CASE", "SM BOX", "SM PACK", "SM PKG"], 1, 5),
-                                    ("Brand#23", ["MED BAG", "MED BOX", "MED PKG", "MED PACK"], 10, 10),
-                                    ("Brand#34", ["LG CASE", "LG BOX", "LG PACK", "LG PKG"], 20, 15)]:
+    for brand, conts, qlo, smax in Q19_BRANCHES:
         conjs.append([(6, "==", B[brand]), (7, "in", [C[c] for c in conts]), (1, ">=", qlo * 100),
                       (1, "<=", (qlo + 10) * 100), (8, ">=", 1), (8, "<=", smax), (4, "in", modes),
                       (5, "==", I_["DELIVER IN PERSON"])])

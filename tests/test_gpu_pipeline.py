@@ -534,16 +534,17 @@ def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel, variant):
     keep, views = load([fk, v])
     dkeep, dviews = load([tv])
     plan = plans.fkjsel(thr, mode)
-    os.environ["VD_FKJS_VARIANT"] = {"gather_fold": "off", "fk_select_sum_ldg": "ldg", "fk_select_sum_tma": "tma"}[variant]
-    try:
+    fk_var = {"gather_fold": "off", "fk_select_sum_ldg": "ldg", "fk_select_sum_tma": "tma"}[variant]
+    with env(VD_FKJS_VARIANT=fk_var, VD_LATE="off"):
         got = vd.decode_partials(run(plan, views, n, dviews, want=(variant.replace("_ldg", "").replace("_tma", ""),))[0],
                                  plan)
-    finally:
-        os.environ.pop("VD_FKJS_VARIANT", None)
-    if not exp_c:
-        assert got == {}
-    else:
-        assert got == {0: [exp_s or 0, exp_c, exp_c]}
+    want = {} if not exp_c else {0: [exp_s or 0, exp_c, exp_c]}
+    assert got == want
+    if variant == "gather_fold" and mode == vd.VD_SEL_BRANCH:
+        # branching without the Fig 16 kernels: the late-materialisation fragment
+        # (v < t is an i32 interval lead; fk and the lookup per qualifying row)
+        with env(VD_FKJS_VARIANT="off"):
+            assert vd.decode_partials(run(plan, views, n, dviews, want=("late",))[0], plan) == want
 
 
 @pytest.mark.parametrize("seed", range(10))
