@@ -1526,17 +1526,6 @@ __device__ __forceinline__ int late_pred_c(const LateLead& ld, int nconj, const 
     return any;
 }
 
-// 16 u8 rows (one 128-bit word) against [lo, hi] per byte -> 16-bit mask
-__device__ __forceinline__ uint32_t lt_mask_u8(int4 v, uint32_t lo4, uint32_t hi4) {
-    const uint32_t w[4] = {(uint32_t)v.x, (uint32_t)v.y, (uint32_t)v.z, (uint32_t)v.w};
-    uint32_t m = 0;
-#pragma unroll
-    for (int i = 0; i < 4; ++i) {
-        const uint32_t r = __vcmpgeu4(w[i], lo4) & __vcmpleu4(w[i], hi4);  // 0xFF per passing byte
-        m |= (((r & 0x01010101u) * 0x01020408u) >> 24) << (4 * i);         // byte k -> bit k
-    }
-    return m;
-}
 __device__ __forceinline__ uint32_t lt_mask_i32(const int4 (&v)[4], int32_t lo, int32_t hi) {
     uint32_t m = 0;
 #pragma unroll
@@ -1633,8 +1622,25 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
         uint32_t m = 0;
         if (q < nq) {
             m = 0xFFFFu;
+            if (N8 > 0) {
+                // byte masks of every u8 lead column ANDed word by word, then
+                // one byte -> bit extraction
+                uint32_t r[4] = {~0u, ~0u, ~0u, ~0u};
 #pragma unroll
-            for (int j = 0; j < N8; ++j) m &= lt_mask_u8(c8[j], ld.lo8[j], ld.hi8[j]);
+                for (int j = 0; j < N8; ++j) {
+                    const uint32_t w[4] = {(uint32_t)c8[j].x, (uint32_t)c8[j].y, (uint32_t)c8[j].z, (uint32_t)c8[j].w};
+                    if (ld.lo8[j] == ld.hi8[j]) {
+#pragma unroll
+                        for (int i = 0; i < 4; ++i) r[i] &= __vcmpeq4(w[i], ld.lo8[j]);
+                    } else {
+#pragma unroll
+                        for (int i = 0; i < 4; ++i) r[i] &= __vcmpgeu4(w[i], ld.lo8[j]) & __vcmpleu4(w[i], ld.hi8[j]);
+                    }
+                }
+                m = 0;
+#pragma unroll
+                for (int i = 0; i < 4; ++i) m |= (((r[i] & 0x01010101u) * 0x01020408u) >> 24) << (4 * i);
+            }
             if (I32) m &= lt_mask_i32(c32, ld.lo32, ld.hi32);
         }
         load_lead(q + wstride, c8, c32);
