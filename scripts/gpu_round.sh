@@ -1,6 +1,6 @@
 # Re-validation of HEAD on a fresh box: smoke, every GPU parity test, the
 # default bench line, every workload's bench line, the launch list, and
-# full ncu captures of the L2-gather fragments (q9, fkjsel).
+# full ncu captures of the L2-gather fragments (q9, q19 late).
 set -x
 mkdir -p gpurun_out
 nvidia-smi --query-gpu=name,clocks.sm,clocks.max.sm,memory.total --format=csv > gpurun_out/nvsmi.txt 2>&1
@@ -15,5 +15,5 @@ timeout 300 python bench.py --workload fkjsel --selectivity 0.5 --no-cpu-baselin
 timeout 300 python bench.py --impl reference --steps 3 --warmup 3 > gpurun_out/bench_ref.json 2>> gpurun_out/bench_misc.err
 timeout 600 ncu --metrics gpu__time_duration.sum --clock-control none -c 60 --csv --log-file gpurun_out/launches_q1.csv python bench.py --steps 3 --warmup 3 --no-cpu-baseline --no-e2e > gpurun_out/ncu_launch.log 2>&1
 timeout 600 ncu --set full --clock-control none --import-source on -k regex:k_pipe_fkg -s 1 -c 1 -o gpurun_out/prof_q9 -f python bench.py --workload q9 --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/ncu_q9.log 2>&1
-timeout 600 ncu --set full --clock-control none -k regex:k_pipe_fkjs -s 1 -c 1 -o gpurun_out/prof_fkjsel -f python bench.py --workload fkjsel --selectivity 0.5 --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/ncu_fkjsel.log 2>&1
+timeout 600 ncu --set full --clock-control none --import-source on -k regex:k_pipe_late -s 1 -c 1 -o gpurun_out/prof_q19 -f python bench.py --workload q19 --steps 1 --warmup 1 --no-cpu-baseline --no-e2e > gpurun_out/ncu_q19.log 2>&1
 ls -la gpurun_out
