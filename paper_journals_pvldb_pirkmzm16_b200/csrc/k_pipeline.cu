@@ -1385,7 +1385,18 @@ struct LateLead {
     // has no such form and the term lists of GfArgs are interpreted instead
     int32_t ncons[VD_MAX_CONJ + 1];
     LtCons cons[VD_MAX_CONJ + 1][VD_MAX_TERMS];
+    // u8 references (up to LT_MAXTAB): their constraints leave cons[] and
+    // become acceptance tables -- tab[k][x] bit c (c < nconj: conjunction c,
+    // bit LT_COMMON: the common terms) = value x (255: epsilon) passes every
+    // constraint of that conjunction on reference tref[k]; tcm[k] = the
+    // conjunctions constraining it.  The predicate becomes an AND of masks.
+    int32_t ntab;
+    int32_t tref[4];
+    uint32_t tcm[4];
+    uint8_t tab[4][256];
 };
+constexpr int LT_MAXTAB = 4;
+constexpr int LT_COMMON = 4;  // = VD_MAX_CONJ
 
 // L2 eviction policy for data re-read by other rows (the dimension lookups).
 __device__ __forceinline__ uint64_t policy_evict_last() {
@@ -1514,16 +1525,30 @@ __device__ __forceinline__ int late_cons(const LtCons* cs, int n, const int64_t 
     return r;
 }
 __device__ __forceinline__ int late_pred_c(const LateLead& ld, int nconj, const int64_t (*sv)[LT_THREADS], int tid,
-                                           uint32_t known) {
-    const int r = late_cons(ld.cons[VD_MAX_CONJ], ld.ncons[VD_MAX_CONJ], sv, tid, known);
-    if (r == 0 || nconj == 0) return r;
-    int any = 0;
-    for (int c = 0; c < nconj; ++c) {
-        const int cj = late_cons(ld.cons[c], ld.ncons[c], sv, tid, known);
-        if (cj == 1) return r;
-        if (cj == 2) any = 2;
+                                           uint32_t known, const uint8_t (*stab)[256]) {
+    const uint32_t conjs = (1u << nconj) - 1;
+    uint32_t m = conjs | (1u << LT_COMMON), und = 0;
+    for (int k = 0; k < ld.ntab; ++k) {
+        const int r = ld.tref[k];
+        if (!((known >> r) & 1u)) {
+            und |= ld.tcm[k];
+            continue;
+        }
+        const int64_t x = sv[r][tid];
+        m &= stab[k][x == INT64_MIN ? 255 : (int)x];
     }
-    return any;
+    // the rest, only for the conjunctions (and common terms) still alive
+    if (!((m >> LT_COMMON) & 1u) || (nconj > 0 && !(m & conjs))) return 0;
+    for (uint32_t live = m; live; live &= live - 1) {
+        const int c = __ffs(live) - 1;
+        const int t = late_cons(ld.cons[c], ld.ncons[c], sv, tid, known);
+        if (t == 0) m &= ~(1u << c);
+        if (t == 2) und |= 1u << c;
+    }
+    if (!((m >> LT_COMMON) & 1u)) return 0;
+    if (nconj > 0 && !(m & conjs)) return 0;
+    const bool yes = !((und >> LT_COMMON) & 1u) && (nconj == 0 || (m & conjs & ~und));
+    return yes ? 1 : 2;
 }
 
 __device__ __forceinline__ uint32_t lt_mask_i32(const int4 (&v)[4], int32_t lo, int32_t hi) {
@@ -1559,7 +1584,10 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
     int64_t(*s_a)[LT_THREADS] = reinterpret_cast<int64_t(*)[LT_THREADS]>(lt_smem + nref * LT_THREADS * 8);
     int32_t(*s_q)[LT_QCAP] = reinterpret_cast<int32_t(*)[LT_QCAP]>(lt_smem + (nref + NA + 1) * LT_THREADS * 8);
     __shared__ int64_t s_acc[LT_THREADS / 32][VD_MAX_AGGS + 1];
+    __shared__ uint8_t s_tab[LT_MAXTAB][256];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31, tid = threadIdx.x;
+    for (int k = 0; k < ld.ntab; ++k) s_tab[k][tid] = ld.tab[k][tid];  // LT_THREADS == 256
+    __syncthreads();
     const uint64_t pol_s = policy_evict_first(), pol_d = policy_evict_last();
     int32_t* q_ = s_q[warp];
     int cnt = 0;  // warp-uniform queue depth
@@ -1568,10 +1596,10 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
     auto fold_row = [&](int64_t row) {
         late_load(a, ld.pref1, row, s_v, tid, pol_s, pol_d);
         const bool compiled = ld.ncons[0] >= 0;
-        int t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1) : late_pred(a, s_v, tid, ld.pref1);
+        int t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1, s_tab) : late_pred(a, s_v, tid, ld.pref1);
         if (t == 2) {
             late_load(a, ld.pref & ~ld.pref1, row, s_v, tid, pol_s, pol_d);
-            t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref) : late_pred(a, s_v, tid, ld.pref);
+            t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref, s_tab) : late_pred(a, s_v, tid, ld.pref);
         }
         if (t != 1) return;
         late_load(a, ld.aref & ~ld.pref, row, s_v, tid, pol_s, pol_d);
@@ -3905,6 +3933,44 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         }
         if (!ok) L.ncons[0] = -1;
         else if (A.pred.nconj == 0) L.ncons[0] = 0;
+        // u8 references: constraints -> acceptance tables (the common terms
+        // sit in row VD_MAX_CONJ = LT_COMMON)
+        auto ref_u8 = [&](int r) { return dtype_of(r) == VD_U8; };
+        L.ntab = 0;
+        if (ok) {
+            for (int c = 0; c <= VD_MAX_CONJ; ++c) {
+                if (c >= A.pred.nconj && c != VD_MAX_CONJ) continue;
+                for (int k = 0; k < L.ncons[c]; ++k) {
+                    const int r = L.cons[c][k].ref;
+                    if (!ref_u8(r)) continue;
+                    int t = -1;
+                    for (int h = 0; h < L.ntab; ++h) t = L.tref[h] == r ? h : t;
+                    if (t < 0 && L.ntab < LT_MAXTAB) {
+                        t = L.ntab++;
+                        L.tref[t] = r;
+                        L.tcm[t] = 0;
+                        std::memset(L.tab[t], 0xFF, 256);
+                    }
+                    if (t < 0) continue;
+                    const LtCons& q = L.cons[c][k];
+                    L.tcm[t] |= 1u << c;
+                    for (int x = 0; x < 256; ++x) {
+                        const bool pass = x != 0xFF && x >= q.lo && x <= q.hi && ((q.in >> (x & 63)) & 1ull);
+                        if (!pass) L.tab[t][x] &= (uint8_t)~(1u << c);
+                    }
+                }
+            }
+            for (int c = 0; c <= VD_MAX_CONJ; ++c) {  // drop the tabulated constraints
+                if (c >= A.pred.nconj && c != VD_MAX_CONJ) continue;
+                int nk = 0;
+                for (int k = 0; k < L.ncons[c]; ++k) {
+                    bool tabbed = false;
+                    for (int h = 0; h < L.ntab; ++h) tabbed = tabbed || L.tref[h] == L.cons[c][k].ref;
+                    if (!tabbed) L.cons[c][nk++] = L.cons[c][k];
+                }
+                L.ncons[c] = nk;
+            }
+        }
         for (int g = 0; g < A.naggs; ++g)
             if (A.a_kind[g] != VD_AGG_COUNT)
                 for (int f = 0; f < A.a_nf[g]; ++f)
