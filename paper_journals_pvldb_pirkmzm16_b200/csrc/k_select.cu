@@ -584,7 +584,23 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
             }
         }
         __syncwarp();
-        for (int k = lane; k < total; k += 32) __stcs(&out[base + k], st[k + (k >> 5)]);
+        // flush: scalar stores up to the first 16-byte boundary of the output
+        // (any 4-byte aligned out_pos), then
+        // one 128-bit streaming store per lane per 128 positions, scalar tail
+        const int h = min(total, (int)(((16 - ((uintptr_t)(out + base) & 15)) & 15) >> 2));
+        if (lane < h) __stcs(&out[base + lane], st[lane]);
+        const int nv = (total - h) >> 2;
+        int4* o4 = reinterpret_cast<int4*>(out + base + h);
+        for (int v = lane; v < nv; v += 32) {
+            const int k = h + 4 * v;
+            int4 q;
+            q.x = st[k + (k >> 5)];
+            q.y = st[k + 1 + ((k + 1) >> 5)];
+            q.z = st[k + 2 + ((k + 2) >> 5)];
+            q.w = st[k + 3 + ((k + 3) >> 5)];
+            __stcs(o4 + v, q);
+        }
+        for (int k = h + 4 * nv + lane; k < total; k += 32) __stcs(&out[base + k], st[k + (k >> 5)]);
         __syncwarp();
     }
 }

@@ -89,6 +89,29 @@ def test_select_f32_single_term_vs_oracle(mode, n):
 
 
 @pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("shift", [1, 2, 3])
+def test_select_into_unaligned_output_vs_oracle(mode, shift):
+    """Positions written to an out_pos that starts 4, 8 or 12 bytes past a
+    16-byte boundary (the position pass's vector flush aligns on the output
+    address), selectivities from sparse to dense, ragged n."""
+    n = 300007
+    v = gen.host(gen.F32_UNIFORM, n, seed=29)
+    dv = cuda_tensor(v)
+    for t in (0.01, 0.5, 0.97):
+        t = float(np.float32(t))
+        pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
+        buf = torch.full((n + 8,), -7, dtype=torch.int32, device="cuda")
+        out = buf[shift:shift + n]
+        cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+        fn = vd.select_branch if mode == "branch" else vd.select_predicated
+        fn([vd.column(dv)], n, vd.pred([[(0, "<", t)]]), out_pos=out, out_count=cnt)
+        c = int(cnt.item())
+        assert c == cnt_o
+        assert np.array_equal(out[:c].cpu().numpy(), pos_o)
+        assert (buf[:shift] == -7).all().item()  # nothing written before out_pos
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
 @pytest.mark.parametrize("dtype", ["u8", "i32", "i64", "f64"])
 @pytest.mark.parametrize("n", [0, 5, 4097, 70001])
 def test_select_dtypes_with_eps_vs_interpreter(mode, dtype, n):
