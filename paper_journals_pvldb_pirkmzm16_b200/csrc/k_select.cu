@@ -543,17 +543,29 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
     int32_t* st = s_stage + warp * (BM_CHUNK + BM_CHUNK / 32);
-    // the next chunk's bitmap word and offset are loaded one iteration ahead,
-    // so their round trip overlaps this chunk's decode and stores
-    uint32_t w_nx = gw < nchunks ? __ldcs(&bits[gw * 32 + lane]) : 0u;
-    int64_t base_nx = gw < nchunks ? __ldcs(&offs[gw]) : 0;
+    // the bitmap words and offsets of the warp's next SW_PF chunks are in
+    // flight while this one is decoded (a register queue shifted each step):
+    // at low selectivity the pass is otherwise one L2/HBM round trip per chunk
+    constexpr int SW_PF = 4;
+    uint32_t wq[SW_PF];
+    int64_t bq[SW_PF];
+#pragma unroll
+    for (int u = 0; u < SW_PF; ++u) {
+        const int64_t cu = gw + u * nw;
+        wq[u] = cu < nchunks ? __ldcs(&bits[cu * 32 + lane]) : 0u;
+        bq[u] = cu < nchunks ? __ldcs(&offs[cu]) : 0;
+    }
     for (int64_t c = gw; c < nchunks; c += nw) {
-        const uint32_t w = w_nx;
-        const int64_t base = base_nx;
-        if (c + nw < nchunks) {
-            w_nx = __ldcs(&bits[(c + nw) * 32 + lane]);
-            base_nx = __ldcs(&offs[c + nw]);
+        const uint32_t w = wq[0];
+        const int64_t base = bq[0];
+#pragma unroll
+        for (int u = 0; u + 1 < SW_PF; ++u) {
+            wq[u] = wq[u + 1];
+            bq[u] = bq[u + 1];
         }
+        const int64_t cn = c + SW_PF * nw;
+        wq[SW_PF - 1] = cn < nchunks ? __ldcs(&bits[cn * 32 + lane]) : 0u;
+        bq[SW_PF - 1] = cn < nchunks ? __ldcs(&offs[cn]) : 0;
         const int pc = __popc(w);
         int incl = pc;
 #pragma unroll
