@@ -8,7 +8,8 @@ times (columns generated in HBM by gen.device, the same fragments).
 - C2 selection over 1e9 f32: the position list is checked through properties
   that determine it uniquely at any size -- strictly increasing, every
   position qualifies, and the count equals the oracle's count.
-- C5 Q9-style FK join at SF12.5 (one GPU's share of SF100 over 8 GPUs).
+- C5 Q9-style FK join at SF12.5 (one GPU's share of SF100 over 8 GPUs) and
+  Q19-style FK join at SF100 (the bench's single-GPU workload).
 """
 import concurrent.futures as cf
 import os
@@ -134,3 +135,46 @@ def test_fkj_q9_sf12p5_exact():
             a0, c0 = exp.get(k, (0, 0))
             exp[k] = (a0 + rv, c0 + c)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+
+
+def q19_codes():
+    return {"brand": {s: i for i, s in enumerate(gen.BRAND)},
+            "container": {s: i for i, s in enumerate(gen.CONTAINER)},
+            "shipmode": {s: i for i, s in enumerate(gen.SHIPMODE)},
+            "shipinstruct": {s: i for i, s in enumerate(gen.SHIPINSTRUCT)}}
+
+
+def test_fkj_q19_sf100_exact():
+    """C5 Q19-style FK join at SF100 (600 M lineitem rows x 20 M part rows),
+    the bench's launch configuration: the late-materialisation fragment by
+    default and the dense star-join fragment (VD_LATE=off) both equal the
+    oracle's brute-force loop over row chunks."""
+    sf = 100.0
+    n = gen.lineitem_rows(sf)
+    cols, views = device_columns(plans.Q19_COLS, n, sf)
+    dcols, dviews = device_columns(plans.Q19_DIMS, gen.part_rows(sf), sf, table=gen.PART_COLS)
+    plan = plans.q19(q19_codes())
+    got, frag = run(plan, views, n, dviews)
+    assert frag == "late"
+    os.environ["VD_LATE"] = "off"
+    try:
+        got_dense, frag_dense = run(plan, views, n, dviews)
+    finally:
+        del os.environ["VD_LATE"]
+    assert frag_dense == "star_join"
+    del cols, dcols
+    supp = {k: gen.host(c, gen.supplier_rows(sf), sf=sf) for k, c in gen.SUPPLIER_COLS.items()}
+    part_cols = {k: gen.host(c, gen.part_rows(sf), sf=sf) for k, c in gen.PART_COLS.items()}
+
+    def part(a, b):
+        li = {k: gen.host(c, b - a, a, sf=sf) for k, c in gen.LINEITEM_COLS.items()}
+        return oracle.fkj(0, li, part_cols, supp)
+
+    exp = {}
+    for r in chunked(n, part, chunk=10_000_000):
+        for k, (rv, c) in r.items():
+            a0, c0 = exp.get(k, (0, 0))
+            exp[k] = (a0 + rv, c0 + c)
+    assert exp and exp[0][1] > 0
+    assert {k: tuple(v[:2]) for k, v in got.items()} == exp
+    assert got_dense == got
