@@ -543,7 +543,7 @@ def test_fkjsel_fig16_strategies_vs_interpreter(mode, sel, variant):
     if variant == "gather_fold" and mode == vd.VD_SEL_BRANCH:
         # branching without the Fig 16 kernels: the late-materialisation fragment
         # (v < t is an i32 interval lead; fk and the lookup per qualifying row)
-        with env(VD_FKJS_VARIANT="off"):
+        with env(VD_FKJS_VARIANT="off", VD_LATE="force"):
             assert vd.decode_partials(run(plan, views, n, dviews, want=("late",))[0], plan) == want
 
 
@@ -612,3 +612,27 @@ def test_late_fragment_random_plans_vs_oracle(seed):
     with env(VD_LATE="force"):
         got = vd.decode_partials(run(plan, views, n, want=("late",))[0], plan)
     assert got == exp
+
+
+def test_late_fragment_selectivity_estimate():
+    """Default dispatch takes the late-materialisation fragment only when the
+    lead intervals are estimated (min/max metadata, even spread) to pass few
+    rows: a 2% lead on an i32 column goes late, a 60% one stays dense
+    (gather-fold); VD_LATE=force takes it regardless.  Same results."""
+    rng = np.random.default_rng(5)
+    n, m = 200003, 5000
+    fk = rng.integers(1, m + 1, n).astype(np.int32)
+    v = rng.integers(0, 1000, n).astype(np.int32)
+    tv = rng.integers(-10**6, 10**6, m).astype(np.int64)
+    keep, views = load([fk, v])
+    dkeep, dviews = load([tv])
+    for thr, frag in ((20, "late"), (600, "gather_fold")):
+        plan = vd.pipeline(pred_=vd.pred([[(1, "<", thr)]]), gathers=[(0, 0, 1)], aggs=[("sum", [2]), ("count",)])
+        sel = v < thr
+        exp = {0: [int(tv[fk[sel] - 1].sum()), int(sel.sum()), int(sel.sum())]}
+        with env(VD_FKJS_VARIANT="off", VD_STAR_VARIANT="off"):
+            got, _ = run(plan, views, n, dviews, want=(frag,))
+            assert vd.decode_partials(got, plan) == exp
+            with env(VD_LATE="force"):
+                got, _ = run(plan, views, n, dviews, want=("late",))
+                assert vd.decode_partials(got, plan) == exp
