@@ -538,11 +538,11 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
                                                           int32_t* __restrict__ out) {
     // stage index k is stored at k + k/32 (one pad word per 32): lanes whose
     // cursors are 32 apart hit different banks
-    __shared__ int32_t s_stage[(BM_THREADS / 32) * (BM_CHUNK + BM_CHUNK / 32)];
+    __shared__ int32_t s_stage[(BM_THREADS / 32) * (BM_CHUNK + BM_CHUNK / 32 + 4)];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int64_t gw = ((int64_t)blockIdx.x * BM_THREADS + threadIdx.x) >> 5;
     const int64_t nw = ((int64_t)gridDim.x * BM_THREADS) >> 5;
-    int32_t* st = s_stage + warp * (BM_CHUNK + BM_CHUNK / 32);
+    int32_t* st = s_stage + warp * (BM_CHUNK + BM_CHUNK / 32 + 4);
     // the bitmap words and offsets of the warp's next SW_PF chunks are in
     // flight while this one is decoded (a register queue shifted each step):
     // at low selectivity the pass is otherwise one L2/HBM round trip per chunk
@@ -576,16 +576,20 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
         const int excl = incl - pc;
         const int total = __shfl_sync(VD_FULL, incl, 31);
         const int32_t row0 = (int32_t)(c * BM_CHUNK + lane * 32);
+        // output index k sits at stage index j = k + a (a = the output's
+        // misalignment in words), physically j + j/32: the 16-byte groups of
+        // the output are 4-word groups of the stage that never straddle a pad
+        const int a = (int)(((uintptr_t)(out + base) >> 2) & 3);
         if (MODE == 0) {
             uint32_t m = w;
-            int k = excl;
+            int k = excl + a;
             while (m) {
                 st[k + (k >> 5)] = row0 + (__ffs(m) - 1);
                 ++k;
                 m &= m - 1;
             }
         } else {
-            int sel = excl, unsel = total + (lane * 32 - excl);
+            int sel = excl + a, unsel = total + (lane * 32 - excl) + a;
 #pragma unroll
             for (int i = 0; i < 32; ++i) {
                 const int f = (w >> i) & 1u;
@@ -599,20 +603,19 @@ __global__ void __launch_bounds__(BM_THREADS) k_sel_write(const uint32_t* __rest
         // flush: scalar stores up to the first 16-byte boundary of the output
         // (any 4-byte aligned out_pos), then
         // one 128-bit streaming store per lane per 128 positions, scalar tail
-        const int h = min(total, (int)(((16 - ((uintptr_t)(out + base) & 15)) & 15) >> 2));
-        if (lane < h) __stcs(&out[base + lane], st[lane]);
+        const int h = min(total, (4 - a) & 3);
+        if (lane < h) __stcs(&out[base + lane], st[lane + a]);  // j < 32: no pad yet
         const int nv = (total - h) >> 2;
         int4* o4 = reinterpret_cast<int4*>(out + base + h);
         for (int v = lane; v < nv; v += 32) {
-            const int k = h + 4 * v;
-            int4 q;
-            q.x = st[k + (k >> 5)];
-            q.y = st[k + 1 + ((k + 1) >> 5)];
-            q.z = st[k + 2 + ((k + 2) >> 5)];
-            q.w = st[k + 3 + ((k + 3) >> 5)];
-            __stcs(o4 + v, q);
+            const int j = h + a + 4 * v;  // a multiple of 4
+            const int32_t* g = st + j + (j >> 5);
+            __stcs(o4 + v, make_int4(g[0], g[1], g[2], g[3]));
         }
-        for (int k = h + 4 * nv + lane; k < total; k += 32) __stcs(&out[base + k], st[k + (k >> 5)]);
+        for (int k = h + 4 * nv + lane; k < total; k += 32) {
+            const int j = k + a;
+            __stcs(&out[base + k], st[j + (j >> 5)]);
+        }
         __syncwarp();
     }
 }
