@@ -636,3 +636,28 @@ def test_late_fragment_selectivity_estimate():
             with env(VD_LATE="force"):
                 got, _ = run(plan, views, n, dviews, want=("late",))
                 assert vd.decode_partials(got, plan) == exp
+
+
+@pytest.mark.parametrize("n", [1, 15, 16, 17, 511, 513, 4099])
+@pytest.mark.parametrize("lead", ["none", "all", "some"])
+def test_late_fragment_edge_sizes(n, lead):
+    """Late fragment at sizes around its 16-row lead words and 32-row drains
+    (tail rows only, one word, one word + tail, partial drains) with leads
+    that pass nothing, everything or some rows; against numpy."""
+    rng = np.random.default_rng(n * 7 + len(lead))
+    m = 300
+    a = rng.integers(0, 4, n).astype(np.uint8)
+    fk = rng.integers(1, m + 1, n).astype(np.int32)
+    x = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    d = rng.integers(0, 10, m).astype(np.uint8)
+    cmp_, val = {"none": ("==", 9), "all": ("<=", 3), "some": ("==", 2)}[lead]
+    plan = vd.pipeline(pred_=vd.pred([[(0, cmp_, val), (3, "<", 5)]]), gathers=[(1, 0, 1)],
+                       aggs=[("sum", [2]), ("count",)])
+    lead_ok = (a == val) if cmp_ == "==" else (a <= val)
+    sel = lead_ok & (d[fk - 1] < 5)
+    exp = {0: [int(x[sel].sum()), int(sel.sum()), int(sel.sum())]} if sel.any() else {}
+    keep, views = load([a, fk, x])
+    dkeep, dviews = load([d])
+    with env(VD_LATE="force"):
+        got, _ = run(plan, views, n, dviews, want=("late",))
+    assert vd.decode_partials(got, plan) == exp
