@@ -4008,13 +4008,12 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         Slot16* parts = (Slot16*)((char*)ws + 256);
         cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+        // (the attribute is per device context: set on every launch, as for
+        // the other dynamic-shared-memory fragments)
 #define LT_GO(N8_, I32_)                                                                                    \
     do {                                                                                                    \
-        static bool attr_ = false;                                                                          \
-        if (!attr_) {                                                                                       \
-            cudaFuncSetAttribute(k_pipe_late<N8_, I32_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
-            attr_ = true;                                                                                   \
-        }                                                                                                   \
+        e = cudaFuncSetAttribute(k_pipe_late<N8_, I32_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }                     \
         k_pipe_late<N8_, I32_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);               \
     } while (0)
         if (n8 == 2) { if (i32) LT_GO(2, true); else LT_GO(2, false); }
