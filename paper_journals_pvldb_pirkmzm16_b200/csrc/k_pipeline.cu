@@ -1630,7 +1630,6 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
         __syncwarp();
     };
     const int64_t nq = a.n / 16;
-    const int64_t wstride = (int64_t)gridDim.x * LT_THREADS;
     // lead words of the current step, and of the next one loaded before the
     // current step's drain (the stream stays in flight behind the late loads)
     int4 c8[N8 > 0 ? N8 : 1], c32[4];
@@ -1643,9 +1642,25 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
             for (int k = 0; k < 4; ++k) w32[k] = lt_ld16(ld.c32 + 16 * q + 4 * k, pol_s);
         }
     };
-    int64_t q0 = (int64_t)blockIdx.x * LT_THREADS + warp * 32;
+    // dynamic work distribution: a warp claims LT_GRAB consecutive 32-word
+    // blocks of the lead at a time from a global counter (done[1]; one
+    // same-address atomic per claim, so claims must be coarse), so no warp
+    // idles at the end while others still drain
+    constexpr unsigned LT_GRAB = 16;
+    unsigned rb = 0, re = 0;  // the warp's claimed block range [rb, re)
+    auto next_block = [&]() -> int64_t {
+        if (rb == re) {
+            unsigned b = 0;
+            if (lane == 0) b = atomicAdd(done + 1, 1u);
+            rb = __shfl_sync(VD_FULL, b, 0) * LT_GRAB;
+            re = rb + LT_GRAB;
+        }
+        return (int64_t)(rb++) * 32;
+    };
+    int64_t q0 = next_block();
     load_lead(q0 + lane, c8, c32);
-    for (; q0 < nq; q0 += wstride) {
+    while (q0 < nq) {
+        const int64_t q1 = next_block();
         const int64_t q = q0 + lane;
         uint32_t m = 0;
         if (q < nq) {
@@ -1671,7 +1686,7 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
             }
             if (I32) m &= lt_mask_i32(c32, ld.lo32, ld.hi32);
         }
-        load_lead(q + wstride, c8, c32);
+        load_lead(q1 + lane, c8, c32);
         // compaction: the lanes' qualifying rows, in row order, onto the warp's queue
         const int pc = __popc(m);
         int incl = pc;
@@ -1687,6 +1702,7 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
         }
         cnt += __shfl_sync(VD_FULL, incl, 31);
         while (cnt >= 32) drain(32);
+        q0 = q1;
     }
     if (cnt > 0) drain(cnt);
     // ragged tail (< 16 rows): warp 0 of block 0, one row per lane
@@ -4006,7 +4022,7 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         const int grid = grid_persistent(per_sm);
         unsigned int* dn = (unsigned int*)ws;
         Slot16* parts = (Slot16*)((char*)ws + 256);
-        cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
+        cudaError_t e = cudaMemsetAsync(dn, 0, 8, s);  // done counter + lead claim counter
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
         // (the attribute is per device context: set on every launch, as for
         // the other dynamic-shared-memory fragments)
