@@ -3908,7 +3908,7 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         }
         if (n8 == 0 && !i32) return VD_OK;
         // a late load per surviving row costs more than streaming the row
-        // past ~20% survivors (Q19 3.6%: 0.76 ms late vs 3.08 ms dense; Q6
+        // past ~20% survivors (Q19 3.6%: 0.69 ms late vs 3.08 ms dense; Q6
         // 15%: 0.28 vs 0.25 ms): by default only clearly selective leads
         if (late_policy() != 2 && est > 0.15) return VD_OK;
         int nc = 0;  // the lead intervals replace the hoisted terms on their columns
