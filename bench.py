@@ -367,6 +367,19 @@ def main():
         looked_up = n if args.sel_mode == "predicated" else sel_rows // max(world, 1)
         alg_bytes = n * bpr + 64 * looked_up
         extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64}
+        if vd.last_fragment() == "late":
+            # late materialisation (A31/A33/A34): fact.v in full, of fact.fk
+            # the 64-byte blocks holding a qualifying row, 64 B per lookup
+            thr = int(round(args.selectivity * plans.FKJSEL_VMAX))
+            mask = cols[1] < thr
+            r = 64 // cols[0].element_size()
+            full = n // r * r
+            fk_blocks = int(mask[:full].view(-1, r).any(1).sum().item()) + int(bool(mask[full:].any().item()))
+            looked_up = int(mask.sum().item())
+            alg_bytes = n * cols[1].element_size() + 64 * fk_blocks + 64 * looked_up
+            extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64,
+                     "fk_blocks": fk_blocks}
+            del mask
     elif w == "q19" and vd.last_fragment() == "late":
         # late-materialisation fragment, readings A31/A33: the lead columns
         # (l_shipmode, l_shipinstruct: the u8 terms every conjunction shares)

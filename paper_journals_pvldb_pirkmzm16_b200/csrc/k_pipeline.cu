@@ -3908,9 +3908,10 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         }
         if (n8 == 0 && !i32) return VD_OK;
         // a late load per surviving row costs more than streaming the row
-        // past ~20% survivors (Q19 3.6%: 0.69 ms late vs 3.08 ms dense; Q6
-        // 15%: 0.28 vs 0.25 ms): by default only clearly selective leads
-        if (late_policy() != 2 && est > 0.15) return VD_OK;
+        // past ~10-20% survivors (Q19 3.6%: 0.69 ms late vs 3.08 ms dense;
+        // Fig 16 10%: 0.55 vs 0.57 ms, 20%: 0.91 vs 0.67 ms; Q6 15%: 0.28 vs
+        // 0.25 ms): by default only clearly selective leads
+        if (late_policy() != 2 && est > 0.12) return VD_OK;
         int nc = 0;  // the lead intervals replace the hoisted terms on their columns
         for (int k = 0; k < A.ncommon; ++k)
             if (!lead[A.common[k].col]) A.common[nc++] = A.common[k];
@@ -4197,13 +4198,15 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         if (st != VD_OK || done) return st;
         st = try_fkg(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
-        st = try_fkjs(p, cols, ncols, n, dims, out, ws, s, nl, &done);
-        if (st != VD_OK || done) return st;
         if (late_policy() == 1) {
-            // branching scalar FK joins (Q19 shape): late loads beat the dense star fragment
+            // branching scalar FK joins with a selective lead: late loads beat
+            // the dense star fragment (Q19) and the per-row selective FK sum
+            // (Fig 16 at s <= 10%: 0.22 vs 0.49 ms at 1%)
             st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done, true);
             if (st != VD_OK || done) return st;
         }
+        st = try_fkjs(p, cols, ncols, n, dims, out, ws, s, nl, &done);
+        if (st != VD_OK || done) return st;
         st = try_star(p, cols, ncols, n, dims, out, ws, s, nl, &done);
         if (st != VD_OK || done) return st;
         st = try_gf(p, cols, ncols, n, dims, out, ws, s, nl, &done);
