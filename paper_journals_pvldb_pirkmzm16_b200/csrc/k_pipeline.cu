@@ -1934,11 +1934,12 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
             for (int k = 0; k < RPT; ++k) key[k] = keyof(pd[k], pkb[k], px[k], py[k], v[k]);
             foldn(key, v);
         };
+        int s = 0;          // ring stage and its phase, advanced without
+        uint32_t ph = 0;    // a division by the runtime stage count
         for (int64_t it = 0;; ++it) {
             const int64_t tile = blockIdx.x + it * gridDim.x;
             if (tile >= ntiles) break;
-            const int s = (int)(it % a.nstages);
-            mbar_wait(&full[s], (uint32_t)((it / a.nstages) & 1));
+            mbar_wait(&full[s], ph);
             const uint8_t* st = smem + (size_t)s * SB;
             int32_t f[RPT], kb[RPT];
             int64_t x[RPT], y[RPT];
@@ -1952,6 +1953,7 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(&empty[s]);
+            if (++s == a.nstages) { s = 0; ph ^= 1u; }
             int d[RPT];
 #pragma unroll
             for (int k = 0; k < RPT; ++k) d[k] = gather(true, f[k]);
