@@ -661,3 +661,78 @@ def test_late_fragment_edge_sizes(n, lead):
     with env(VD_LATE="force"):
         got, _ = run(plan, views, n, dviews, want=("late",))
     assert vd.decode_partials(got, plan) == exp
+
+
+@pytest.mark.parametrize("seed", range(12))
+def test_late_fragment_random_fk_plans_vs_oracle(seed):
+    """Late fragment with FK lookups on random branching plans: a common u8
+    lead on the fact table, per-conjunction terms on two u8 dimension columns
+    (acceptance tables: every comparison kind, IN sets, NE, codes >= 64), an
+    i32 dimension column and an i64 fact column (constraints), epsilon in
+    every column and FKs outside the dimension; against the oracle (one
+    FoldSelect program per conjunction through Gather, union, then
+    Gather -> Multiply -> FoldSum / FoldCount)."""
+    rng = np.random.default_rng(900 + seed)
+    n, m = 60001 + 31 * seed, 2503
+    fk = rng.integers(-3, m + 5, n).astype(np.int32)
+    ld = rng.integers(0, 6, n).astype(np.uint8)
+    rq = rng.integers(0, 6000, n).astype(np.int64)
+    x = rng.integers(0, 10**7, n).astype(np.int64)
+    d1 = rng.integers(0, 80, m).astype(np.uint8)
+    d2 = rng.integers(0, 40, m).astype(np.uint8)
+    dr = rng.integers(1, 51, m).astype(np.int32)
+    eps = {}
+    for nm, arr, e in [("fk", fk, -2**31), ("ld", ld, 255), ("rq", rq, -2**63), ("x", x, -2**63),
+                       ("d1", d1, 255), ("d2", d2, 255), ("dr", dr, -2**31)]:
+        msk = rng.random(arr.size) < 0.01
+        arr[msk] = e
+        eps[nm] = msk
+    ref_idx = {"fk": 0, "ld": 1, "rq": 2, "x": 3, "d1": 4, "d2": 5, "dr": 6}
+
+    def rand_term(k):
+        if k in ("d1", "d2"):
+            cmp = str(rng.choice([">", "<", "==", ">=", "<=", "!=", "in"]))
+            if cmp == "in":
+                return k, cmp, sorted(set(int(v) for v in rng.integers(0, 64, rng.integers(1, 12))))
+            return k, cmp, int(rng.integers(0, 90))
+        hi = 6000 if k == "rq" else 50
+        return k, str(rng.choice([">", "<", ">=", "<="])), int(rng.integers(0, hi))
+
+    lead = ("ld", "==", int(rng.integers(0, 6)))  # ~1/6 of the rows: a selective lead
+    conjs = []
+    for _ in range(int(rng.integers(1, 4))):
+        names = [k for k in ("d1", "d2", "dr", "rq") if rng.random() < 0.5] or ["d1"]
+        conjs.append([lead] + [rand_term(k) for k in names])
+    sel = np.zeros(n, dtype=bool)
+    inputs = {f"fact__{k}": (v, eps[k]) for k, v in (("fk", fk), ("ld", ld), ("rq", rq))}
+    inputs.update({f"dim__{k}": (v, eps[k]) for k, v in (("d1", d1), ("d2", d2), ("dr", dr))})
+    oref = {"ld": "fact.ld", "rq": "fact.rq", "d1": "gd1", "d2": "gd2", "dr": "gdr"}
+    for terms in conjs:
+        lines = ["p := Subtract(fact.fk, 1)", "gd1 := Gather(dim.d1, p)", "gd2 := Gather(dim.d2, p)",
+                 "gdr := Gather(dim.dr, p)"]
+        names = []
+        for j, (k, cmp, val) in enumerate(terms):
+            _term_expr(f"t{j}", oref[k], cmp, val, lines)
+            names.append(f"t{j}")
+        lines.append(f"q := LogicalAnd({names[0]}, {names[0]})")
+        for nm in names[1:]:
+            lines.append(f"q := LogicalAnd(q, {nm})")
+        lines.append("pos := FoldSelect(q)")
+        pos, pe = oracle.run("\n".join(lines), **inputs).get_arrays("pos")
+        sel[pos[~pe]] = True
+    upos = np.nonzero(sel)[0].astype(np.int64)
+    agg = oracle.run("""
+    gx := Gather(fact.x, pos)
+    s := FoldSum(gx)
+    c := FoldCount(pos)
+    """, fact__x=(x, eps["x"]), pos=upos)
+    exp = {0: [int(agg.get("s")[0]), int(agg.get("c")[0]), int(agg.get("c")[0])]} if upos.size else {}
+    keep, views = load([fk, ld, rq, x])
+    dkeep, dviews = load([d1, d2, dr])
+    plan = vd.pipeline(pred_=vd.pred([[(ref_idx[k], cmp, val) for k, cmp, val in t] for t in conjs]),
+                       gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)], aggs=[("sum", [3]), ("count",)])
+    with env(VD_LATE="force"):
+        got = vd.decode_partials(run(plan, views, n, dviews, want=("late",))[0], plan)
+    assert got == exp
+    with env(VD_LATE="off", VD_STAR_VARIANT="off"):  # the dense gather-fold fragment agrees
+        assert vd.decode_partials(run(plan, views, n, dviews, want=("gather_fold",))[0], plan) == got
