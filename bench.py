@@ -431,7 +431,7 @@ def main():
                      "frac": achieved / peak, "peak_kind": peak_kind,
                      "traffic": ncu_traffic(f"fkjsel_s{args.selectivity:g}_{args.sel_mode}" if w == "fkjsel" else w),
                      "bytes_per_row": alg_bytes / n if n else bpr,
-                     "kernel": "k_pipe_q1+k_q1_remap" if w == "q1" and not args.generic else "vd_run_pipeline",
+                     "kernel": "k_pipe_q1_tma" if w == "q1" and not args.generic else "vd_run_pipeline",
                      "kernel_ms": kernel_ms, **extra},
         "clocks": clk,
         "e2e": e2e,
