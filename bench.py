@@ -34,8 +34,8 @@ METRIC = "rows/s and achieved HBM GB/s (% of peak) for TPC-H Q1/Q6 at 1/2/4/8 B2
 
 # Algorithmic bytes per row: every
 # column each query reads, once.
-BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "q19": 4 + 3 * 8 + 1 + 1,
-                 "q9": 4 + 4 + 2 * 8, "fkjsel": 4 + 4}
+BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "selpos": 4, "c1": 4,
+                 "q19": 4 + 3 * 8 + 1 + 1, "q9": 4 + 4 + 2 * 8, "fkjsel": 4 + 4, "q15": 24}
 L2_CAP_BYTES_PER_CLK = 6300  # B300_MICROARCH.md "LTS throughput cap" (full chip)
 
 
@@ -46,7 +46,8 @@ def parse():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
     ap.add_argument("--workload", default="q1",
-                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14", "q15"])
+                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14", "q15",
+                             "c1"])
     ap.add_argument("--chunk", type=int, default=0,
                     help="select_unfused: rows per materialised chunk (0 = whole table; Fig 15 'Vectorized')")
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
@@ -83,13 +84,31 @@ def hbm_peak():
         return 6650.0, "fallback"
 
 
-def ncu_traffic(workload):
+NOMINAL_HBM_GBS = 8000.0  # B200 HBM3e nominal (report beside the measured peak)
+
+
+def hbm_roofline(achieved, kernel, kernel_ms, traffic=None, **extra):
+    """`roofline` object for an HBM-bound kernel: achieved algorithmic GB/s
+    against the measured copy peak (MEASURED_PEAKS.json) and, beside it, the
+    nominal 8 TB/s."""
+    peak, kind = hbm_peak()
+    return {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+            "peak_kind": kind, "peak_nominal": NOMINAL_HBM_GBS, "frac_nominal": achieved / NOMINAL_HBM_GBS,
+            "traffic": traffic, "kernel": kernel, "kernel_ms": kernel_ms, **extra}
+
+
+def ncu_traffic(workload, world=1):
     """dram bytes per launch of the dominant kernel from the committed
-    `ncu --set full` summary (profiles/ncu_summary.json), else None."""
+    `ncu --set full` summary (profiles/ncu_summary.json), else None.  The
+    capture is of the single-GPU launch; a rank of an N-GPU run scans a
+    1/N row range, so its per-launch traffic is the capture's / N (the
+    streamed columns dominate; replicated dimension tables are a small
+    constant)."""
     try:
         with open(os.path.join(ROOT, "profiles", "ncu_summary.json")) as f:
             d = json.load(f)
-        return d.get(workload, {}).get("dram_bytes_per_launch")
+        t = d.get(workload, {}).get("dram_bytes_per_launch")
+        return None if t is None else t / max(world, 1)
     except Exception:
         return None
 
@@ -153,47 +172,164 @@ class ClockSampler:
 # ---------------------------------------------------------------------------
 # CPU oracle baseline (bounded sample)
 # ---------------------------------------------------------------------------
-def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5):
-    """Time the oracle as it stands (the literal Voodoo interpreter, one
-    thread) on chunks of the same workload until ~budget_s of CPU work."""
+def host_info():
+    """CPU model string and host RAM (SURVEY §8(d) timing protocol)."""
+    model, ram = None, None
+    try:
+        with open("/proc/cpuinfo") as f:
+            for ln in f:
+                if ln.startswith("model name"):
+                    model = ln.split(":", 1)[1].strip()
+                    break
+    except OSError:
+        pass
+    try:
+        with open("/proc/meminfo") as f:
+            for ln in f:
+                if ln.startswith("MemTotal"):
+                    ram = round(int(ln.split()[1]) / 2**20, 1)
+                    break
+    except OSError:
+        pass
+    return {"cpu_model": model, "host_ram_gib": ram, "hardware_concurrency": os.cpu_count()}
+
+
+def oracle_task(workload, sf, seed, sel_t):
+    """(make(row0, m) -> inputs, run(inputs) -> partial, merge(a, b), what):
+    the oracle program of each workload over one row range.  Partials
+    decompose over row ranges (pin P8), so a partitioned run merges them."""
     import numpy as np
 
     import gen
     import oracle
     from oracle import programs
 
-    chunk = 1 << 19
-    rows_done, t_total = 0, 0.0
-    row0 = 0
-    n_total = gen.lineitem_rows(sf) if workload != "select" else 10**9
-    while t_total < budget_s and row0 < n_total:
-        m = min(chunk, n_total - row0)
+    def add_dict(a, b):
+        out = dict(a)
+        for k, v in b.items():
+            out[k] = [x + y for x, y in zip(out[k], v)] if k in out else list(v)
+        return out
+
+    def add_tuple(a, b):
+        return tuple(x + y for x, y in zip(a, b))
+
+    if workload in ("select", "selpos"):
+        def make(row0, m):
+            return gen.host(gen.F32_UNIFORM, m, row0, seed=seed)
         if workload == "select":
-            v = gen.host(gen.F32_UNIFORM, m, row0, seed=seed)
-            t0 = time.perf_counter()
-            p = oracle.Program()
-            p.set("input.val", v)
-            p.run(programs.SELECT_SUM.format(intent=m, t=float(np.float32(sel_t)).hex()))
-            t_total += time.perf_counter() - t0
-        else:
-            li = {k: gen.host(c, m, row0, sf=sf, seed=seed) for k, c in gen.LINEITEM_COLS.items()}
-            t0 = time.perf_counter()
+            def run(v):
+                p = oracle.Program()
+                p.set("input.val", v)
+                p.run(programs.SELECT_SUM.format(intent=v.size, t=float(np.float32(sel_t)).hex()))
+                return (float(p.get("totalSum")[0] or 0.0), int(p.get("count")[0] or 0))
+            return make, run, add_tuple, "literal Voodoo interpreter, SELECT_SUM program (Fig 8 shape)"
+
+        def run(v):
+            return (oracle.select_f32(v, float(np.float32(sel_t)), "lt")[1],)
+        return make, run, add_tuple, "brute-force selection loop -> int32 positions (oracle/tpch_oracle.cpp)"
+
+    names = {"q1": plans_cols("Q1_COLS"), "q6": plans_cols("Q6_COLS"), "q15": ["l_shipdate", "l_suppkey",
+             "l_extendedprice", "l_discount"]}.get(workload, list(gen.LINEITEM_COLS))
+
+    def make(row0, m):
+        return {k: gen.host(gen.LINEITEM_COLS[k], m, row0, sf=sf, seed=seed) for k in names}
+
+    if workload == "q1":
+        def run(li):
             p = oracle.Program()
             for k, v in li.items():
                 p.set("lineitem." + k, v)
-            if workload == "q1":
-                p.run(programs.Q1.format(ship_max_p1=10472))
-            elif workload == "q6":
-                p.run(programs.Q6.format(intent=1 << 30, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
-            else:
-                oracle.q1(li)  # FKJ: brute-force layer (interpreter needs a calendar dim)
-            t_total += time.perf_counter() - t0
+            p.run(programs.Q1.format(ship_max_p1=10472))
+            keys = p.get("o_key")
+            outs = [p.get(o) for o in programs.Q1_OUTPUTS]
+            return {k: [o[j] for o in outs] for j, k in enumerate(keys) if k is not None}
+        return make, run, add_dict, "literal Voodoo interpreter, Q1 program (Fig 10/11 shape)"
+    if workload == "q6":
+        def run(li):
+            p = oracle.Program()
+            for k, v in li.items():
+                p.set("lineitem." + k, v)
+            p.run(programs.Q6.format(intent=1 << 30, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
+            return (int(p.get("revenue")[0] or 0), int(p.get("count")[0] or 0))
+        return make, run, add_tuple, "literal Voodoo interpreter, Q6 program (Fig 8 shape)"
+    if workload == "q15":
+        def run(li):
+            return {k: list(v) for k, v in oracle.q15(li).items()}
+        return make, run, add_dict, "brute-force Q15 revenue-view loop (oracle/tpch_oracle.cpp)"
+    # FK joins (C5): the brute-force join loop over the replicated dimension tables
+    part = {k: gen.host(c, gen.part_rows(sf), sf=sf, seed=seed) for k, c in gen.PART_COLS.items()}
+    supp = {k: gen.host(c, gen.supplier_rows(sf), sf=sf, seed=seed) for k, c in gen.SUPPLIER_COLS.items()}
+    variant = 0 if workload == "q19" else 1
+
+    def run(li):
+        return {k: list(v) for k, v in oracle.fkj(variant, li, part, supp).items()}
+    return make, run, add_dict, f"brute-force {workload.upper()}-style FK join loop (oracle/tpch_oracle.cpp)"
+
+
+def plans_cols(name):
+    from paper_journals_pvldb_pirkmzm16_b200 import plans
+    return list(getattr(plans, name))
+
+
+def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5, n_total=None, partitioned=True):
+    """Time the oracle as it stands on a bounded sample of the workload:
+    single-threaded over row chunks until ~budget_s of CPU work, then (SURVEY
+    §8(d)) the same rows partitioned over N = hardware_concurrency threads,
+    thread i interpreting rows [i*S/N, (i+1)*S/N) (the Fig 3 control vector,
+    P:L241-250) and the partials merged.  Input generation is excluded."""
+    import concurrent.futures as cf
+
+    import gen
+
+    if workload == "fkjsel":
+        return None
+    make, run, merge, what = oracle_task(workload, sf, seed, sel_t)
+    chunk = 1 << 19
+    if n_total is None:
+        n_total = gen.lineitem_rows(sf) if workload not in ("select", "selpos") else 10**9
+    rows_done, t_total, row0, res1 = 0, 0.0, 0, None
+    while t_total < budget_s and row0 < n_total:
+        m = min(chunk, n_total - row0)
+        x = make(row0, m)
+        t0 = time.perf_counter()
+        r = run(x)
+        t_total += time.perf_counter() - t0
+        res1 = r if res1 is None else merge(res1, r)
         rows_done += m
         row0 += m
-    return {"value": rows_done / t_total, "unit": "rows/s", "cores": 1, "kind": "oracle",
-            "sample": f"{rows_done} rows of the {workload} workload (rows 0..{rows_done - 1}, chunks of {chunk}), "
-                      f"literal Voodoo interpreter (oracle/voodoo_oracle.cpp), {t_total:.1f} s single-threaded",
-            "seconds": t_total}
+    out = {"value": rows_done / t_total, "unit": "rows/s", "cores": 1, "kind": "oracle",
+           "sample": f"{rows_done} rows of the {workload} workload (rows 0..{rows_done - 1}, chunks of {chunk}), "
+                     f"{what}, {t_total:.1f} s single-threaded",
+           "seconds": t_total, **host_info()}
+    if partitioned and rows_done > 0:
+        N = os.cpu_count() or 1
+        bounds = [(i * rows_done // N, (i + 1) * rows_done // N) for i in range(N)]
+        sub = 1 << 17
+        work = [[make(a0, min(sub, b0 - a0)) for a0 in range(a, b, sub)] for a, b in bounds]
+
+        def thread(items):  # ctypes releases the GIL inside the C oracle
+            acc = None
+            for x in items:
+                r = run(x)
+                acc = r if acc is None else merge(acc, r)
+            return acc
+
+        t0 = time.perf_counter()
+        with cf.ThreadPoolExecutor(N) as ex:
+            parts = list(ex.map(thread, work))
+        dt = time.perf_counter() - t0
+        resN = None
+        for r in parts:
+            if r is not None:
+                resN = r if resN is None else merge(resN, r)
+        same = resN == res1 if workload != "select" else (
+            abs(resN[0] - res1[0]) <= 1e-9 * abs(res1[0]) and resN[1] == res1[1])
+        out["partitioned"] = {"value": rows_done / dt, "unit": "rows/s", "threads": N, "seconds": dt,
+                              "merged_equals_single_thread": bool(same),
+                              "sample": f"the same {rows_done} rows, thread i -> rows [i*S/N, (i+1)*S/N) "
+                                        f"(Fig 3 control vector), sub-chunks of {sub}, partials merged"}
+        del work
+    return out
 
 
 # ---------------------------------------------------------------------------
@@ -216,6 +352,8 @@ def main():
         return fig14_main(args, rank, world, local)
     if args.workload == "q15":
         return q15_main(args, rank, world, local, sf)
+    if args.workload == "c1":
+        return c1_main(args, rank, world, local)
 
     import torch
     import torch.distributed as dist
@@ -416,23 +554,13 @@ def main():
         "vs_baseline": None,
         "dtype": "f32/f64" if w == "select" else "int64",
         "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
-        "config": {
-            "workload": {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
-                         "q9": f"fkj_q9_sf{sf:g}", "select": f"select_f32_{n_total}_s{args.selectivity:g}",
-                         "fkjsel": f"fkjsel_{n_total}x{plans.FKJSEL_TARGET_ROWS}_s{args.selectivity:g}"}[w],
-            "rows": n_total, "rows_per_gpu": n, "sf": sf, "sel_mode": args.sel_mode,
-            "fragment": "generic" if args.generic else vd.last_fragment(),
-            "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
-            "l2": f"inputs {n * bpr / 1e9:.1f} GB per GPU > 126 MB L2: no flush needed",
-            "seed": args.seed,
-        },
+        "config": bench_config(args, w, sf, world),
+        "fragment": "generic" if args.generic else vd.last_fragment(),
         "hbm_gbs": achieved,
-        "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                     "frac": achieved / peak, "peak_kind": peak_kind,
-                     "traffic": ncu_traffic(f"fkjsel_s{args.selectivity:g}_{args.sel_mode}" if w == "fkjsel" else w),
-                     "bytes_per_row": alg_bytes / n if n else bpr,
-                     "kernel": "k_pipe_q1_tma" if w == "q1" and not args.generic else "vd_run_pipeline",
-                     "kernel_ms": kernel_ms, **extra},
+        "roofline": hbm_roofline(
+            achieved, "k_pipe_q1_tma" if w == "q1" and not args.generic else "vd_run_pipeline", kernel_ms,
+            ncu_traffic(f"fkjsel_s{args.selectivity:g}_{args.sel_mode}" if w == "fkjsel" else w, world),
+            bytes_per_row=alg_bytes / n if n else bpr, **extra),
         "clocks": clk,
         "e2e": e2e,
         "gpu_launches": launches_per_step * steps,
@@ -442,8 +570,9 @@ def main():
         "wall_s": wall,
     }
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
-        line["cpu_baseline"] = cpu_baseline(w, sf if w != "select" else 0, args.seed, args.cpu_seconds,
-                                            args.selectivity)
+        cb = cpu_baseline(w, sf, args.seed, args.cpu_seconds, args.selectivity, n_total)
+        if cb is not None:
+            line["cpu_baseline"] = cb
     if rank == 0:
         print(json.dumps(line), flush=True)
     comm.close()
@@ -506,13 +635,104 @@ def selpos_main(args, rank, world, local):
     line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
             "vs_baseline": None, "dtype": "f32", "data": "synthetic (f32 U[0,1), gen/vd_gen.h)",
-            "config": {"workload": f"selpos_f32_{n_total}_s{args.selectivity:g}", "sel_mode": args.sel_mode,
-                       "selected": c, "achieved_selectivity": c / n,
-                       "l2": f"input {4 * n / 1e9:.1f} GB > 126 MB L2: no flush needed"},
-            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
-                         "peak_kind": kind, "traffic": ncu_traffic(f"selpos_s{args.selectivity:g}_{args.sel_mode}"),
-                         "kernel": "k_select", "kernel_ms": ms},
+            "config": bench_config(args, "selpos", 0.0, world),
+            "selected": c, "achieved_selectivity": c / n,
+            "roofline": hbm_roofline(alg, "k_sel_* (bitmap + scan + positions)", ms,
+                                     ncu_traffic(f"selpos_s{args.selectivity:g}_{args.sel_mode}", world)),
             "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cb = cpu_baseline("selpos", 0.0, args.seed, args.cpu_seconds, args.selectivity, n_total)
+        if cb is not None:
+            line["cpu_baseline"] = cb
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    comm.close()
+
+
+def c1_main(args, rank, world, local):
+    """C1 (BASELINE.json configs[0]): 2^20 f32 U[0,1), v < 0.5, branching vs
+    predicated: the position list (vd_select_*, Fig 1) plus the FoldSum of
+    the selected values (the fused selective-sum fragment, Fig 8/15).  The
+    4 MiB input is L2-resident by design, so the HBM roofline does not
+    apply: per-call microseconds are reported warm (back to back) and cold
+    (each call after a 512 MB write that evicts L2), on the launching stream
+    with CUDA events.  A step = positions + sum, both modes reported; the
+    line's value is the warm branching step.  Each rank runs an independent
+    replica (C1 does not shard: 'replicas only')."""
+    import numpy as np
+    import torch
+
+    import gen
+    import oracle
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+
+    ndev = torch.cuda.device_count()
+    torch.cuda.set_device(local % ndev)
+    dev = torch.device("cuda", local % ndev)
+    comm = Comm(world, args.dist_backend, dev)
+    stream = torch.cuda.current_stream()
+    n = args.rows or (1 << 20)
+    v = torch.empty(n, dtype=torch.float32, device=dev)
+    gen.device(gen.F32_UNIFORM, v.data_ptr(), n, 0, seed=args.seed, stream=stream.cuda_stream)
+    t = float(np.float32(args.selectivity))
+    col = [vd.column(v)]
+    p = vd.pred([[(0, "<", t)]])
+    pos = torch.empty(n, dtype=torch.int32, device=dev)
+    cnt = torch.zeros(1, dtype=torch.int64, device=dev)
+    ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_SELECT, n), dev)
+    flush = torch.empty(512 << 20, dtype=torch.uint8, device=dev)
+    res = {}
+    launches = 0
+    steps = args.steps or 200
+    for mode in ("branch", "predicated"):
+        sel = vd.select_predicated if mode == "predicated" else vd.select_branch
+        plan = plans.selsum(t, vd.VD_SEL_PREDICATED if mode == "predicated" else vd.VD_SEL_BRANCH)
+        out = torch.empty(vd.partials_bytes(plan), dtype=torch.uint8, device=dev)
+        pws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
+        calls = {"positions": lambda: sel(col, n, p, out_pos=pos, out_count=cnt, ws=ws, stream=stream),
+                 "sum": lambda: vd.run_pipeline(plan, col, n, out=out, ws=pws, stream=stream)}
+        for _ in range(max(args.warmup, 3)):
+            for f in calls.values():
+                f()
+        torch.cuda.synchronize()
+        r = {}
+        for cold in (False, True):
+            for name, f in list(calls.items()) + [("step", lambda: [g() for g in calls.values()])]:
+                ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
+                      for _ in range(steps)]
+                for i in range(steps):
+                    if cold:
+                        flush.fill_(i & 0xFF)  # evict L2 (126 MB) before the call
+                    ev[i][0].record(stream)
+                    f()
+                    ev[i][1].record(stream)
+                torch.cuda.synchronize()
+                us = sorted(a.elapsed_time(b) * 1e3 for a, b in ev)
+                r[f"{name}_{'cold' if cold else 'warm'}_us"] = {"median": statistics.median(us), "best": us[0]}
+        launches += vd.last_launch_count()
+        # parity with the oracle (count, positions, f64 sum within 1e-9)
+        c = int(cnt.item())
+        pos_o, cnt_o, (sh, sl) = oracle.select_f32(v.cpu().numpy(), t, "lt")
+        got = vd.decode_partials(out.cpu().numpy().tobytes(), plan, float_aggs=[True])[0]
+        r["parity"] = bool(c == cnt_o and np.array_equal(pos[:c].cpu().numpy(), pos_o) and got[1] == cnt_o
+                           and abs(got[0] - (sh + sl)) <= 1e-9 * abs(sh + sl))
+        r["selected"] = c
+        res[mode] = r
+    ms = comm.max([res["branch"]["step_warm_us"]["median"] / 1e3])[0]
+    line = {"metric": METRIC, "value": n * world / (ms * 1e-3), "unit": "rows/s", "n_gpus": world,
+            "steps": steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "f32/f64", "data": "synthetic (f32 U[0,1), gen/vd_gen.h)",
+            "config": bench_config(args, "c1", 0.0, world),
+            "c1": res,
+            "roofline": {"bound": "latency", "achieved": None, "peak": None, "unit": "us", "frac": None,
+                         "traffic": None, "kernel": "k_sel_* + k_pipe_selsum_tma",
+                         "note": "4 MiB input + 2 MiB positions are L2-resident: launch/latency-bound by design "
+                                 "(SURVEY §8(d) C1); the HBM roofline applies to C2, not here"},
+            "clocks": None, "e2e": None, "gpu_launches": launches * steps}
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
+        cb = cpu_baseline("select", 0.0, args.seed, min(args.cpu_seconds, 5.0), args.selectivity, n)
+        if cb is not None:
+            line["cpu_baseline"] = cb
     if rank == 0:
         print(json.dumps(line), flush=True)
     comm.close()
@@ -856,14 +1076,15 @@ def q15_main(args, rank, world, local, sf):
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
             "vs_baseline": None, "dtype": "int64",
             "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
-            "config": {"workload": f"tpch_q15_revenue_sf{sf:g}", "rows": n, "groups_domain": D, "groups": g,
-                       "sf": sf, "l2": f"inputs {n * 24 / 1e9:.1f} GB > 126 MB L2: no flush needed",
-                       "seed": args.seed},
-            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
-                         "peak_kind": kind, "traffic": ncu_traffic("q15"),
-                         "bytes_per_row": alg_bytes / n, "dense_bytes_per_row": 24, "selectivity": sel,
-                         "kernel": "vd_group_fold (k_grp_init + k_grp_fold + compaction)", "kernel_ms": ms},
+            "config": bench_config(args, "q15", sf, 1), "groups_domain": D, "groups": g,
+            "roofline": hbm_roofline(alg, "vd_group_fold (k_grp_init + k_grp_fold + compaction)", ms,
+                                     ncu_traffic("q15"), bytes_per_row=alg_bytes / n, dense_bytes_per_row=24,
+                                     selectivity=sel),
             "clocks": clk, "e2e": None, "gpu_launches": launches * steps, "result_digest": digest}
+    if not args.no_cpu_baseline:
+        cb = cpu_baseline("q15", sf, args.seed, args.cpu_seconds, args.selectivity, n)
+        if cb is not None:
+            line["cpu_baseline"] = cb
     print(json.dumps(line), flush=True)
 
 
@@ -897,7 +1118,7 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
         vcols = []
         for h, d, v in zip(host, dst, views):
             c = vd.load_column(h, d, compute_minmax=False, stream=stream)
-            c.min, c.max, c.has_minmax = v.min, v.max, v.has_minmax  # catalog metadata
+            c.min, c.max, c.has_minmax, c.flags = v.min, v.max, v.has_minmax, v.flags  # catalog metadata
             vcols.append(c)
         vd.run_pipeline(plan, vcols, n, dim_views, out=out, ws=ws, stream=stream)
         res.copy_(out, non_blocking=True)
@@ -910,6 +1131,36 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
             "pinned": pinned, "reps": reps, "s_per_step": dt}
 
 
+def workload_rows(args, w, sf):
+    import gen
+    if w in ("select", "selpos", "select_unfused"):
+        return args.rows or 10**9
+    if w in ("fkjsel", "fig14"):
+        return args.rows or 200_000_000
+    if w == "c1":
+        return args.rows or (1 << 20)
+    return gen.lineitem_rows(sf)
+
+
+def bench_config(args, w, sf, world):
+    """The workload's `config` (identical in the GPU arm and the reference
+    arm: the driver compares them)."""
+    n_total = workload_rows(args, w, sf)
+    bpr = BYTES_PER_ROW.get(w, 4)
+    name = {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
+            "q9": f"fkj_q9_sf{sf:g}", "q15": f"tpch_q15_revenue_sf{sf:g}",
+            "select": f"select_f32_{n_total}_s{args.selectivity:g}",
+            "selpos": f"selpos_f32_{n_total}_s{args.selectivity:g}",
+            "c1": f"c1_select_f32_{n_total}_s{args.selectivity:g}",
+            "fkjsel": f"fkjsel_{n_total}x16777216_s{args.selectivity:g}"}.get(w, w)
+    per_gpu = n_total // world
+    return {"workload": name, "rows": n_total, "rows_per_gpu": per_gpu, "sf": sf, "sel_mode": args.sel_mode,
+            "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
+            "l2": ("inputs L2-resident by design (C1): warm and cold (after a 512 MB L2 flush) reported"
+                   if w == "c1" else f"inputs {per_gpu * bpr / 1e9:.1f} GB per GPU > 126 MB L2: no flush needed"),
+            "seed": args.seed}
+
+
 def reference_arm(args, rank, world, sf):
     """The tier's reference arm: the CPU oracle on the same config/metric."""
     if rank != 0:
@@ -919,20 +1170,22 @@ def reference_arm(args, rank, world, sf):
     budget = max(1.0, min(args.cpu_seconds, 60.0) / max(steps, 1))
     vals = []
     cb = None
+    n_total = workload_rows(args, w, sf)
     if args.warmup > 0:
-        cpu_baseline(w, sf if w != "select" else 0, args.seed, 0.5, args.selectivity)
+        cpu_baseline(w, sf, args.seed, 0.5, args.selectivity, n_total, partitioned=False)
     t0 = time.perf_counter()
     for _ in range(steps):
-        cb = cpu_baseline(w, sf if w != "select" else 0, args.seed, budget, args.selectivity)
+        cb = cpu_baseline(w, sf, args.seed, budget, args.selectivity, n_total, partitioned=False)
         vals.append(cb["value"])
     wall = time.perf_counter() - t0
     v = statistics.median(vals)
     line = {"metric": METRIC, "value": v, "unit": "rows/s", "impl": "reference", "n_gpus": world, "steps": steps,
             "warmup": args.warmup, "ms_per_step": wall / steps * 1e3, "higher_is_better": True, "scaling": "strong",
-            "vs_baseline": None, "dtype": "int64", "data": "synthetic",
-            "config": {"workload": {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
-                                    "q9": f"fkj_q9_sf{sf:g}", "select": "select_f32"}[w], "sf": sf},
-            "cpu_baseline": {"value": v, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": cb["sample"]},
+            "vs_baseline": None, "dtype": "f32/f64" if w in ("select", "selpos", "c1") else "int64",
+            "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, host)",
+            "config": bench_config(args, w, sf, world),
+            "cpu_baseline": {"value": v, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": cb["sample"],
+                             **host_info()},
             "e2e": {"value": v, "unit": "rows/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
 

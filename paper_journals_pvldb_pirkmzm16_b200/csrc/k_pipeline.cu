@@ -383,36 +383,70 @@ struct Q1Acc {
     int64_t s0[G], s1[G], s2[G], s3[G], dc[G];
 };
 
-template <int G, bool NARROW>
-__device__ __forceinline__ void q1_row(Q1Acc<G, NARROW>& A, const Q1Args& a, bool pass, int key, int64_t v0,
-                                       int64_t v1, int64_t v2, int64_t v3) {
-    int64_t dp, ch;
+// Q1 row values (V0, V1, dp, ch, disc|count word).  EPS (some referenced
+// column lacks VD_COL_NOEPS): an epsilon operand makes each product that
+// uses it epsilon, and an epsilon value is skipped by its SUM (readings A5,
+// A9) -- it contributes 0 while the row still counts (COUNT(*) = the row
+// count, as the generic fragment).  Without EPS the metadata has proven
+// that no referenced slot is epsilon.
+struct Q1Vals {
+    int64_t v0, v1, dp, ch, dc;
+};
+template <bool NARROW, bool EPS>
+__device__ __forceinline__ Q1Vals q1_vals(const Q1Args& a, int64_t v0, int64_t v1, int64_t v2, int64_t v3) {
+    Q1Vals r;
     if (NARROW) {
         // metadata proves |V1|, |a1+b1*V2|, |dp|, |a2+b2*V3| < 2^31 and the
         // constants fit in 32 bits: the factors are exact in wrapping 32-bit
         // arithmetic and each product is one 32x32->64 IMAD.WIDE
         int32_t f1 = (int32_t)a.a1 + (int32_t)a.b1 * (int32_t)v2;
-        dp = (int64_t)(int32_t)v1 * (int64_t)f1;
+        r.dp = (int64_t)(int32_t)v1 * (int64_t)f1;
         int32_t f2 = (int32_t)a.a2 + (int32_t)a.b2 * (int32_t)v3;
-        ch = (int64_t)(int32_t)dp * (int64_t)f2;
+        r.ch = (int64_t)(int32_t)r.dp * (int64_t)f2;
     } else {
-        dp = v1 * (a.a1 + a.b1 * v2);
-        ch = dp * (a.a2 + a.b2 * v3);
+        r.dp = v1 * (a.a1 + a.b1 * v2);
+        r.ch = r.dp * (a.a2 + a.b2 * v3);
     }
-    const int64_t dc = v2 + (1ll << Q1_CSHIFT);
+    if (EPS) {
+        const bool e0 = v0 == INT64_MIN, e1 = v1 == INT64_MIN, e2 = v2 == INT64_MIN, e3 = v3 == INT64_MIN;
+        r.v0 = e0 ? 0 : v0;
+        r.v1 = e1 ? 0 : v1;
+        if (e1 | e2) r.dp = 0;
+        if (e1 | e2 | e3) r.ch = 0;
+        r.dc = (e2 ? 0 : v2) + (1ll << Q1_CSHIFT);
+    } else {
+        r.v0 = v0;
+        r.v1 = v1;
+        r.dc = v2 + (1ll << Q1_CSHIFT);
+    }
+    return r;
+}
+
+// key of a row from its two dictionary codes; -1 if either code is epsilon
+// (0xFF: the key is epsilon, the row has no group -- Partition drops it, A9)
+template <bool EPS>
+__device__ __forceinline__ int q1_key(const Q1Args& a, uint32_t c1, uint32_t c2) {
+    if (EPS && (c1 == 0xFFu || c2 == 0xFFu)) return -1;
+    return (int)c1 * a.m1 + (int)c2 * a.m2 + a.koff;
+}
+
+template <int G, bool NARROW, bool EPS>
+__device__ __forceinline__ void q1_row(Q1Acc<G, NARROW>& A, const Q1Args& a, bool pass, int key, int64_t v0,
+                                       int64_t v1, int64_t v2, int64_t v3) {
+    const Q1Vals r = q1_vals<NARROW, EPS>(a, v0, v1, v2, v3);
 #pragma unroll
     for (int g = 0; g < G; ++g) {
         if (pass && key == g) {
-            A.s0[g] += v0;
-            A.s1[g] += v1;
-            A.s2[g] += dp;
-            A.s3[g] += ch;
-            A.dc[g] += dc;
+            A.s0[g] += r.v0;
+            A.s1[g] += r.v1;
+            A.s2[g] += r.dp;
+            A.s3[g] += r.ch;
+            A.dc[g] += r.dc;
         }
     }
 }
 
-template <int G, bool NARROW>
+template <int G, bool NARROW, bool EPS>
 __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant__ Q1Args a, Slot16* __restrict__ parts,
                                                            unsigned int* __restrict__ done, Slot16* __restrict__ out,
                                                            const Q1Map map) {
@@ -446,12 +480,12 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
 #pragma unroll
             for (int j = 0; j < 4; ++j) {
                 bool pass = dd[j] >= a.dlo && dd[j] <= a.dhi;
-                int key = (int)((k1[u] >> (8 * j)) & 0xFF) * a.m1 + (int)((k2[u] >> (8 * j)) & 0xFF) * a.m2 + a.koff;
+                int key = q1_key<EPS>(a, (k1[u] >> (8 * j)) & 0xFF, (k2[u] >> (8 * j)) & 0xFF);
                 int64_t v0 = (j & 1) ? x[u][0][j >> 1].y : x[u][0][j >> 1].x;
                 int64_t v1 = (j & 1) ? x[u][1][j >> 1].y : x[u][1][j >> 1].x;
                 int64_t v2 = (j & 1) ? x[u][2][j >> 1].y : x[u][2][j >> 1].x;
                 int64_t v3 = (j & 1) ? x[u][3][j >> 1].y : x[u][3][j >> 1].x;
-                q1_row<G, NARROW>(A, a, pass, key, v0, v1, v2, v3);
+                q1_row<G, NARROW, EPS>(A, a, pass, key, v0, v1, v2, v3);
             }
         }
     }
@@ -469,12 +503,12 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
 #pragma unroll
         for (int j = 0; j < 4; ++j) {
             bool pass = dd[j] >= a.dlo && dd[j] <= a.dhi;
-            int key = (int)((k1 >> (8 * j)) & 0xFF) * a.m1 + (int)((k2 >> (8 * j)) & 0xFF) * a.m2 + a.koff;
+            int key = q1_key<EPS>(a, (k1 >> (8 * j)) & 0xFF, (k2 >> (8 * j)) & 0xFF);
             int64_t v0 = (j & 1) ? x[0][j >> 1].y : x[0][j >> 1].x;
             int64_t v1 = (j & 1) ? x[1][j >> 1].y : x[1][j >> 1].x;
             int64_t v2 = (j & 1) ? x[2][j >> 1].y : x[2][j >> 1].x;
             int64_t v3 = (j & 1) ? x[3][j >> 1].y : x[3][j >> 1].x;
-            q1_row<G, NARROW>(A, a, pass, key, v0, v1, v2, v3);
+            q1_row<G, NARROW, EPS>(A, a, pass, key, v0, v1, v2, v3);
         }
     }
     // ragged tail (n % 4 rows): thread 0 of the grid
@@ -482,8 +516,8 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
         for (int64_t r = a.nquads * 4; r < a.n; ++r) {
             int dd = a.d[r];
             bool pass = dd >= a.dlo && dd <= a.dhi;
-            int key = (int)a.k1[r] * a.m1 + (int)a.k2[r] * a.m2 + a.koff;
-            q1_row<G, NARROW>(A, a, pass, key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
+            int key = q1_key<EPS>(a, a.k1[r], a.k2[r]);
+            q1_row<G, NARROW, EPS>(A, a, pass, key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
         }
     }
 
@@ -557,30 +591,22 @@ __host__ __device__ constexpr size_t q1t_smem(int G) {
     return (size_t)Q1T_STAGES * Q1T_STAGE_BYTES + (size_t)(G + 1) * Q1T_WORDS * Q1T_NT * 8 + 2 * Q1T_STAGES * 8;
 }
 
-template <bool NARROW>
+template <bool NARROW, bool EPS>
 __device__ __forceinline__ void q1_row_smem(int64_t* __restrict__ acc_t, const Q1Args& a, int G, int32_t dd,
                                             int key, int64_t v0, int64_t v1, int64_t v2, int64_t v3) {
-    const bool pass = dd >= a.dlo && dd <= a.dhi;
-    const int kk = pass ? key : G;  // trash slot for rows that fail the predicate
-    int64_t dp, ch;
-    if (NARROW) {
-        int32_t f1 = (int32_t)a.a1 + (int32_t)a.b1 * (int32_t)v2;
-        dp = (int64_t)(int32_t)v1 * (int64_t)f1;
-        int32_t f2 = (int32_t)a.a2 + (int32_t)a.b2 * (int32_t)v3;
-        ch = (int64_t)(int32_t)dp * (int64_t)f2;
-    } else {
-        dp = v1 * (a.a1 + a.b1 * v2);
-        ch = dp * (a.a2 + a.b2 * v3);
-    }
+    // dlo > INT32_MIN (planner), so an epsilon ship date never passes (A9)
+    const bool pass = dd >= a.dlo && dd <= a.dhi && (!EPS || key >= 0);
+    const int kk = pass ? key : G;  // trash slot for rows that fail the predicate or have no group
+    const Q1Vals r = q1_vals<NARROW, EPS>(a, v0, v1, v2, v3);
     int64_t* p = acc_t + (size_t)kk * Q1T_WORDS * Q1T_NT;
-    p[0 * Q1T_NT] += v0;
-    p[1 * Q1T_NT] += v1;
-    p[2 * Q1T_NT] += dp;
-    p[3 * Q1T_NT] += ch;
-    p[4 * Q1T_NT] += v2 + (1ll << Q1_CSHIFT);
+    p[0 * Q1T_NT] += r.v0;
+    p[1 * Q1T_NT] += r.v1;
+    p[2 * Q1T_NT] += r.dp;
+    p[3 * Q1T_NT] += r.ch;
+    p[4 * Q1T_NT] += r.dc;
 }
 
-template <int G, bool NARROW>
+template <int G, bool NARROW, bool EPS>
 __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_constant__ Q1Args a, int64_t ntiles,
                                                                 Slot16* __restrict__ parts,
                                                                 unsigned int* __restrict__ done,
@@ -648,17 +674,17 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
             if (lane == 0) mbar_arrive(&empty[s]);
 #pragma unroll
             for (int h = 0; h < 2; ++h) {
-                const int key0 = (int)(kk1[h] & 0xFF) * a.m1 + (int)(kk2[h] & 0xFF) * a.m2 + a.koff;
-                const int key1 = (int)(kk1[h] >> 8) * a.m1 + (int)(kk2[h] >> 8) * a.m2 + a.koff;
-                q1_row_smem<NARROW>(acc_t, a, G, dd[h].x, key0, x[h][0].x, x[h][1].x, x[h][2].x, x[h][3].x);
-                q1_row_smem<NARROW>(acc_t, a, G, dd[h].y, key1, x[h][0].y, x[h][1].y, x[h][2].y, x[h][3].y);
+                const int key0 = q1_key<EPS>(a, kk1[h] & 0xFF, kk2[h] & 0xFF);
+                const int key1 = q1_key<EPS>(a, kk1[h] >> 8, kk2[h] >> 8);
+                q1_row_smem<NARROW, EPS>(acc_t, a, G, dd[h].x, key0, x[h][0].x, x[h][1].x, x[h][2].x, x[h][3].x);
+                q1_row_smem<NARROW, EPS>(acc_t, a, G, dd[h].y, key1, x[h][0].y, x[h][1].y, x[h][2].y, x[h][3].y);
             }
         }
         // ragged tail: rows past the last full tile, CTA 0 only
         if (blockIdx.x == 0) {
             for (int64_t r = ntiles * Q1T_TILE + threadIdx.x; r < a.n; r += Q1T_NT) {
-                const int key = (int)a.k1[r] * a.m1 + (int)a.k2[r] * a.m2 + a.koff;
-                q1_row_smem<NARROW>(acc_t, a, G, a.d[r], key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
+                const int key = q1_key<EPS>(a, a.k1[r], a.k2[r]);
+                q1_row_smem<NARROW, EPS>(acc_t, a, G, a.d[r], key, a.v[0][r], a.v[1][r], a.v[2][r], a.v[3][r]);
             }
         }
     }
@@ -755,8 +781,19 @@ constexpr int SC_THREADS = 256;
 
 // MODE 0 branching (late loads: a later column is loaded only for rows whose
 // earlier filters passed), MODE 1 predicated (all loads, contribution x p).
-template <int MODE, bool HAS_F1, bool HAS_F2, bool HAS_VB, typename F0, typename F1, typename F2, typename VA,
-          typename VB>
+// EPS: a value column may hold epsilon (no VD_COL_NOEPS and not a filter
+// column, whose interval already excludes it): an epsilon factor makes the
+// row's value epsilon, skipped by the SUM (A5) while the row still counts.
+template <bool EPS, bool HAS_VB, typename VA, typename VB, typename ACC>
+__device__ __forceinline__ ACC scalar_value(VA va, VB vb) {
+    ACC v = (ACC)va;
+    if (HAS_VB) v *= (ACC)vb;
+    if (EPS && (Eps<VA>::is(va) || (HAS_VB && Eps<VB>::is(vb)))) v = (ACC)0;
+    return v;
+}
+
+template <int MODE, bool EPS, bool HAS_F1, bool HAS_F2, bool HAS_VB, typename F0, typename F1, typename F2,
+          typename VA, typename VB>
 __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constant__ ScalarArgs<F0, F1, F2, VA, VB> a,
                                                             Slot16* __restrict__ parts, unsigned int* __restrict__ done,
                                                             Slot16* __restrict__ out, const ScalarMap map) {
@@ -812,8 +849,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constan
             const bool pj = (p >> j) & 1;
             if (MODE == 0 && !pj) continue;
             VA va = (a.va == (const VA*)a.f0) ? (VA)x0[j] : __ldg(a.va + 4 * q + j);
-            ACC v = (ACC)va;
-            if (HAS_VB) v *= (ACC)__ldg(a.vb + 4 * q + j);
+            const ACC v = scalar_value<EPS, HAS_VB, VA, VB, ACC>(va, HAS_VB ? __ldg(a.vb + 4 * q + j) : VB(1));
             if (MODE == 1) { sum += pj ? v : (ACC)0; cnt += pj; }
             else { sum += v; cnt += 1; }
         }
@@ -824,9 +860,7 @@ __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constan
             if (HAS_F1) pj = pj && ftest(a.f1[r], 1, a.lo, a.hi, a.fcmp, a.fc);
             if (HAS_F2) pj = pj && ftest(a.f2[r], 2, a.lo, a.hi, a.fcmp, a.fc);
             if (!pj) continue;
-            ACC v = (ACC)a.va[r];
-            if (HAS_VB) v *= (ACC)a.vb[r];
-            sum += v;
+            sum += scalar_value<EPS, HAS_VB, VA, VB, ACC>(a.va[r], HAS_VB ? a.vb[r] : VB(1));
             cnt += 1;
         }
     }
@@ -911,7 +945,8 @@ __device__ __forceinline__ T role_ldg(const ScalarTmaArgs& a, int role, int64_t 
     return reinterpret_cast<const T*>(a.col[a.role[role]])[r];
 }
 
-template <int MODE, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA, typename VB>
+template <int MODE, bool EPS, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA,
+          typename VB>
 __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid_constant__ ScalarTmaArgs a,
                                                                     int64_t ntiles, Slot16* __restrict__ parts,
                                                                     unsigned int* __restrict__ done,
@@ -936,8 +971,7 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
         bool p = ftest(x0, 0, a.lo, a.hi, a.fcmp, a.fc);
         if (NF > 1) p = p && ftest(x1, 1, a.lo, a.hi, a.fcmp, a.fc);
         if (NF > 2) p = p && ftest(x2, 2, a.lo, a.hi, a.fcmp, a.fc);
-        ACC v = (ACC)va;
-        if (HVB) v *= (ACC)vb;
+        const ACC v = scalar_value<EPS, HVB, VA, VB, ACC>(va, vb);
         if (MODE == 1) {  // predicated: contribution x predicate
             sum += p ? v : (ACC)0;
             cnt += p;
@@ -2683,6 +2717,40 @@ static int grid_persistent(int per_sm) { return num_sms() * per_sm; }
 // ---- Q1 matching ---------------------------------------------------------
 static bool plain_col(const vd_factor& f) { return f.col >= 0 && f.a == 0 && f.b == 1; }
 
+// Rows one warp of the Q1 fragment folds into its int64 accumulators (the
+// bound the overflow proof needs), for the launch shape that runs:
+//   TMA: `grid` CTAs x Q1T_CW consumer warps; tile t goes to CTA t % grid and
+//        each warp takes 128 rows of it; CTA 0 also folds the ragged tail
+//        (< Q1T_TILE rows over Q1T_NT threads: <= 4 rows per thread);
+//   LDG: `grid` x Q1_THREADS threads striding over quads (4 rows); thread 0
+//        also folds the n % 4 tail rows.
+static double q1_rows_per_warp(bool tma, int64_t n, int grid) {
+    if (tma) {
+        const int64_t ntiles = n / Q1T_TILE;
+        const int64_t tiles_per_cta = (ntiles + grid - 1) / grid;
+        return (double)tiles_per_cta * 128.0 + 32.0 * 4.0;
+    }
+    const int64_t threads = (int64_t)grid * Q1_THREADS;
+    const int64_t nquads = n / 4;
+    return ((double)((nquads + threads - 1) / threads) * 4.0) * 32.0 + 3.0;
+}
+
+template <bool NARROW, bool EPS>
+static cudaError_t launch_q1(int G, bool use_tma, const Q1Args& qa, int64_t ntiles, int tgrid, int grid,
+                             Slot16* parts, unsigned* dn, Slot16* out, const Q1Map& map, cudaStream_t s) {
+#define Q1_LAUNCH(GG)                                                                                         \
+    if (use_tma) {                                                                                            \
+        cudaFuncSetAttribute(k_pipe_q1_tma<GG, NARROW, EPS>, cudaFuncAttributeMaxDynamicSharedMemorySize,      \
+                             (int)q1t_smem(GG));                                                              \
+        k_pipe_q1_tma<GG, NARROW, EPS><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, out, map); \
+    } else {                                                                                                  \
+        k_pipe_q1<GG, NARROW, EPS><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, out, map);                       \
+    }
+    if (G == 4) { Q1_LAUNCH(4) } else if (G == 6) { Q1_LAUNCH(6) } else { Q1_LAUNCH(8) }
+#undef Q1_LAUNCH
+    return cudaGetLastError();
+}
+
 static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, void* out, void* ws,
                         cudaStream_t s, int* nl, bool* done) {
     *done = false;
@@ -2718,7 +2786,9 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
         }
     }
     if (dcol < 0) return VD_OK;  // need a predicate column for this fragment
-    lo = std::max<int64_t>(lo, INT32_MIN);
+    // INT32_MIN is epsilon: a term over epsilon is false (A9), so the
+    // interval never includes it (a one-sided `<=` filter would otherwise)
+    lo = std::max<int64_t>(lo, (int64_t)INT32_MIN + 1);
     hi = std::min<int64_t>(hi, INT32_MAX);
     // aggregates -> raw slots; roles V0..V3
     int V[4] = {-1, -1, -1, -1};
@@ -2771,10 +2841,21 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
     int anycol = -1;
     for (int r = 0; r < 4; ++r) if (V[r] >= 0) anycol = V[r];
     if (anycol < 0) anycol = -2;
-    // overflow proof: per-thread int64 over rows_per_thread rows, warp sums too
-    int grid = grid_persistent(2);
-    int64_t threads = (int64_t)grid * Q1_THREADS;
-    double rows_per_warp = std::ceil((double)n / (double)threads) * 32.0 + 64.0;
+    // launch shape: the TMA variant (num_sms() CTAs x Q1T_NT consumer
+    // threads, 1D bulk copies need every column 16-byte aligned) or the LDG
+    // variant (grid_persistent(2) x Q1_THREADS, 4-row vector loads)
+    auto al = [](const void* q, size_t a) { return ((uintptr_t)q % a) == 0; };
+    const char* var = getenv("VD_Q1_VARIANT");
+    const bool al_all = al(cols[dcol].data, 16) && al(cols[p->key[0].col].data, 16) &&
+                        al(cols[p->key[1].col].data, 16);
+    const bool use_tma = al_all && !(var && strcmp(var, "ldg") == 0);
+    const int64_t ntiles = n / Q1T_TILE;
+    const int tgrid = num_sms();
+    const int grid = grid_persistent(2);
+    // overflow proof: each thread folds its rows into int64 slots and the warp
+    // sums them in int64 (then int128 above), so the bound is rows per WARP of
+    // the variant that launches
+    const double rows_per_warp = q1_rows_per_warp(use_tma, n, use_tma ? tgrid : grid);
     Bound bv[4];
     for (int r = 0; r < 4; ++r) {
         int c = V[r] >= 0 ? V[r] : (anycol >= 0 ? anycol : -1);
@@ -2795,8 +2876,13 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
                   amax(bv[2]) < 2147483647.0 && amax(bv[3]) < 2147483647.0 && fits32(a1) && fits32(b1) &&
                   fits32(a2) && fits32(b2);
     // alignment for the vector loads
-    auto al = [](const void* q, size_t a) { return ((uintptr_t)q % a) == 0; };
     if (!al(cols[dcol].data, 16) || !al(cols[p->key[0].col].data, 4) || !al(cols[p->key[1].col].data, 4)) return VD_OK;
+    // per-row epsilon checks unless the metadata rules epsilon out of every
+    // referenced column (VD_COL_NOEPS)
+    bool eps = !(cols[dcol].flags & VD_COL_NOEPS) || !(cols[p->key[0].col].flags & VD_COL_NOEPS) ||
+               !(cols[p->key[1].col].flags & VD_COL_NOEPS);
+    for (int r = 0; r < 4; ++r)
+        if (V[r] >= 0 && !(cols[V[r]].flags & VD_COL_NOEPS)) eps = true;
     Q1Args qa;
     qa.d = (const int32_t*)cols[dcol].data;
     qa.dlo = (int32_t)lo;
@@ -2822,29 +2908,15 @@ static vd_status try_q1(const vd_pipeline* p, const vd_column* cols, int ncols, 
     Slot16* raw = parts + (size_t)grid * G * 6;
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-    const char* var = getenv("VD_Q1_VARIANT");
-    // 1D bulk copies need 16-byte aligned sources: every column, including the u8 keys
-    const bool al_all = al(cols[p->key[0].col].data, 16) && al(cols[p->key[1].col].data, 16);
-    const bool use_tma = al_all && !(var && strcmp(var, "ldg") == 0);
-    const int64_t ntiles = n / Q1T_TILE;
-    const int tgrid = num_sms();
-#define Q1_LAUNCH(GG)                                                                                          \
-    if (use_tma) {                                                                                             \
-        if (narrow) {                                                                                          \
-            cudaFuncSetAttribute(k_pipe_q1_tma<GG, true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
-            k_pipe_q1_tma<GG, true><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, (Slot16*)out, map);           \
-        } else {                                                                                               \
-            cudaFuncSetAttribute(k_pipe_q1_tma<GG, false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)q1t_smem(GG)); \
-            k_pipe_q1_tma<GG, false><<<tgrid, Q1T_THREADS, q1t_smem(GG), s>>>(qa, ntiles, parts, dn, (Slot16*)out, map);          \
-        }                                                                                                      \
-    } else if (narrow) {                                                                                       \
-        k_pipe_q1<GG, true><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, (Slot16*)out, map);                                   \
-    } else {                                                                                                   \
-        k_pipe_q1<GG, false><<<grid, Q1_THREADS, 0, s>>>(qa, parts, dn, (Slot16*)out, map);                                  \
+    if (narrow) {
+        if (eps) e = launch_q1<true, true>(G, use_tma, qa, ntiles, tgrid, grid, parts, dn, (Slot16*)out, map, s);
+        else e = launch_q1<true, false>(G, use_tma, qa, ntiles, tgrid, grid, parts, dn, (Slot16*)out, map, s);
+    } else {
+        if (eps) e = launch_q1<false, true>(G, use_tma, qa, ntiles, tgrid, grid, parts, dn, (Slot16*)out, map, s);
+        else e = launch_q1<false, false>(G, use_tma, qa, ntiles, tgrid, grid, parts, dn, (Slot16*)out, map, s);
     }
-    if (G == 4) { Q1_LAUNCH(4) } else if (G == 6) { Q1_LAUNCH(6) } else { Q1_LAUNCH(8) }
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     set_fragment(use_tma ? "q1_tma" : "q1_ldg");
-#undef Q1_LAUNCH
     *nl += 1;
     (void)raw;
     e = cudaGetLastError();
@@ -3048,7 +3120,8 @@ static bool scalar_tma_args(const void* const role_ptr[5], const int role_esz[5]
     return (size_t)off * t->nstages + 2 * t->nstages * 8 <= 220 * 1024;
 }
 
-template <int MODE, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA, typename VB>
+template <int MODE, bool EPS, int NF, bool HVB, int TILE, typename F0, typename F1, typename F2, typename VA,
+          typename VB>
 static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* out, const ScalarMap& m,
                                      cudaStream_t s, int* nl) {
     int grid = num_sms();
@@ -3058,7 +3131,7 @@ static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* 
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) return e;
     size_t smem = (size_t)ta.stage_bytes * ta.nstages + 2 * ta.nstages * 8;
-    auto kern = k_pipe_scalar_tma<MODE, NF, HVB, TILE, F0, F1, F2, VA, VB>;
+    auto kern = k_pipe_scalar_tma<MODE, EPS, NF, HVB, TILE, F0, F1, F2, VA, VB>;
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
     kern<<<grid, SCT_THREADS, smem, s>>>(ta, ta.n / TILE, parts, dn, out, m);
     (void)raw;
@@ -3066,7 +3139,8 @@ static cudaError_t launch_scalar_tma(const ScalarTmaArgs& ta, void* ws, Slot16* 
     return cudaGetLastError();
 }
 
-template <int MODE, bool HF1, bool HF2, bool HVB, typename F0, typename F1, typename F2, typename VA, typename VB>
+template <int MODE, bool EPS, bool HF1, bool HF2, bool HVB, typename F0, typename F1, typename F2, typename VA,
+          typename VB>
 static cudaError_t launch_scalar(const ScalarArgs<F0, F1, F2, VA, VB>& sa, void* ws, Slot16* out, const ScalarMap& m,
                                  cudaStream_t s, int* nl) {
     int grid = grid_persistent(4);
@@ -3075,10 +3149,27 @@ static cudaError_t launch_scalar(const ScalarArgs<F0, F1, F2, VA, VB>& sa, void*
     Slot16* raw = parts + (size_t)grid * 2;
     cudaError_t e = cudaMemsetAsync(dn, 0, 4, s);
     if (e != cudaSuccess) return e;
-    k_pipe_scalar<MODE, HF1, HF2, HVB, F0, F1, F2, VA, VB><<<grid, SC_THREADS, 0, s>>>(sa, parts, dn, out, m);
+    k_pipe_scalar<MODE, EPS, HF1, HF2, HVB, F0, F1, F2, VA, VB><<<grid, SC_THREADS, 0, s>>>(sa, parts, dn, out, m);
     (void)raw;
     *nl += 1;
     return cudaGetLastError();
+}
+
+// Rows one consumer thread of the scalar fragment folds into its int64 sum,
+// the larger over the two launch shapes:
+//   TMA: num_sms() CTAs x SCT_NT consumer threads, TILE/SCT_NT rows of each
+//        of the CTA's tiles (tile t -> CTA t % grid), + the ragged tail on
+//        CTA 0 (< TILE rows: <= TILE/SCT_NT per thread); TILE = 2048 (the
+//        i64 value shape);
+//   LDG: grid_persistent(4) x SC_THREADS threads striding over quads, + the
+//        n % 4 tail on thread 0.
+static double scalar_rows_per_thread(int64_t n) {
+    const int64_t TILE = 2048, grid = num_sms();
+    const int64_t ntiles = n / TILE;
+    const double tma = (double)((ntiles + grid - 1) / grid) * (double)(TILE / SCT_NT) + (double)(TILE / SCT_NT);
+    const int64_t threads = (int64_t)grid_persistent(4) * SC_THREADS, nq = n / 4;
+    const double ldg = (double)((nq + threads - 1) / threads) * 4.0 + 3.0;
+    return std::max(tma, ldg);
 }
 
 static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, void* out, void* ws,
@@ -3128,6 +3219,23 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
     }
     if (va < 0) va = fcol[0];
     if (va < 0) return VD_OK;
+    // a term over epsilon is false (A9): integer intervals never include the
+    // type's epsilon (INT_MIN; a one-sided `<` filter would otherwise)
+    for (int j = 0; j < nf; ++j) {
+        if (cols[fcol[j]].dtype == VD_I32) lo[j] = std::max<int64_t>(lo[j], (int64_t)INT32_MIN + 1);
+        else if (cols[fcol[j]].dtype == VD_I64) lo[j] = std::max<int64_t>(lo[j], INT64_MIN + 1);
+        else if (cols[fcol[j]].dtype == VD_U8) hi[j] = std::min<int64_t>(hi[j], 0xFE);
+        else if (cols[fcol[j]].dtype != VD_F32 && cols[fcol[j]].dtype != VD_F64) return VD_OK;
+    }
+    // value columns that may hold epsilon: not proven epsilon-free by the
+    // metadata and not a filter column (whose test already rejects epsilon)
+    auto may_eps = [&](int c) {
+        if (c < 0 || (cols[c].flags & VD_COL_NOEPS)) return false;
+        for (int j = 0; j < nf; ++j)
+            if (fcol[j] == c) return false;
+        return true;
+    };
+    const bool veps = may_eps(va) || may_eps(vb);
     int t0 = nf > 0 ? cols[fcol[0]].dtype : -1;
     int t1 = nf > 1 ? cols[fcol[1]].dtype : -1;
     int t2 = nf > 2 ? cols[fcol[2]].dtype : -1;
@@ -3140,8 +3248,9 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
         Bound B = vb >= 0 ? col_bound(p, cols, ncols, nullptr, vb) : Bound{true, 1, 1};
         if (!A.known || !B.known) return VD_OK;
         double mx = std::max(std::fabs(A.lo), std::fabs(A.hi)) * std::max(std::fabs(B.lo), std::fabs(B.hi));
-        double rows = std::ceil((double)n / ((double)grid_persistent(4) * SC_THREADS)) + 8;
-        if (mx * rows >= 9.0e18) return VD_OK;
+        // per-thread int64 sum: rows one thread folds in the variant that
+        // launches (the larger of the two, the choice is made below)
+        if (mx * scalar_rows_per_thread(n) >= 9.0e18) return VD_OK;
     }
     cudaError_t e = cudaSuccess;
     Slot16* o = (Slot16*)out;
@@ -3170,12 +3279,16 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
             ta.fcmp[0] = ta.fcmp[1] = -1;
             ta.fc[0] = ta.fc[1] = 0;
             ta.n = n;
-            if (mode) e = launch_scalar_tma<1, 3, true, 2048, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
-            else e = launch_scalar_tma<0, 3, true, 2048, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl);
+#define SC_Q6_TMA(M, E) launch_scalar_tma<M, E, 3, true, 2048, int32_t, int64_t, int64_t, int64_t, int64_t>(ta, ws, o, m, s, nl)
+            if (mode) e = veps ? SC_Q6_TMA(1, true) : SC_Q6_TMA(1, false);
+            else e = veps ? SC_Q6_TMA(0, true) : SC_Q6_TMA(0, false);
+#undef SC_Q6_TMA
             set_fragment("scalar_tma");
         } else {
-            if (mode) e = launch_scalar<1, true, true, true>(sa, ws, o, m, s, nl);
-            else e = launch_scalar<0, true, true, true>(sa, ws, o, m, s, nl);
+            if (mode) e = veps ? launch_scalar<1, true, true, true, true>(sa, ws, o, m, s, nl)
+                               : launch_scalar<1, false, true, true, true>(sa, ws, o, m, s, nl);
+            else e = veps ? launch_scalar<0, true, true, true, true>(sa, ws, o, m, s, nl)
+                          : launch_scalar<0, false, true, true, true>(sa, ws, o, m, s, nl);
             set_fragment("scalar_ldg");
         }
     } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && va == fcol[0] && al16(cols[va].data) && use_tma &&
@@ -3223,12 +3336,16 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
             ta.fcmp[0] = fcmp[0]; ta.fcmp[1] = fcmp[1];
             ta.fc[0] = fc[0]; ta.fc[1] = fc[1];
             ta.n = n;
-            if (mode) e = launch_scalar_tma<1, 1, false, 8192, float, float, float, float, float>(ta, ws, o, m, s, nl);
-            else e = launch_scalar_tma<0, 1, false, 8192, float, float, float, float, float>(ta, ws, o, m, s, nl);
+#define SC_F_TMA(M, E) launch_scalar_tma<M, E, 1, false, 8192, float, float, float, float, float>(ta, ws, o, m, s, nl)
+            if (mode) e = veps ? SC_F_TMA(1, true) : SC_F_TMA(1, false);
+            else e = veps ? SC_F_TMA(0, true) : SC_F_TMA(0, false);
+#undef SC_F_TMA
             set_fragment("scalar_tma");
         } else {
-            if (mode) e = launch_scalar<1, false, false, false>(sa, ws, o, m, s, nl);
-            else e = launch_scalar<0, false, false, false>(sa, ws, o, m, s, nl);
+            if (mode) e = veps ? launch_scalar<1, true, false, false, false>(sa, ws, o, m, s, nl)
+                               : launch_scalar<1, false, false, false, false>(sa, ws, o, m, s, nl);
+            else e = veps ? launch_scalar<0, true, false, false, false>(sa, ws, o, m, s, nl)
+                          : launch_scalar<0, false, false, false, false>(sa, ws, o, m, s, nl);
             set_fragment("scalar_ldg");
         }
     } else {

@@ -1,7 +1,7 @@
 """Parity at BASELINE.json's full sizes, in the launch configuration bench.py
 times (columns generated in HBM by gen.device, the same fragments).
 
-- C4 Q1 SF100 (600 M rows) and C3 Q6 SF10 (60 M rows): exact, against the
+- C4 Q1 SF100 (600 M rows), C3 Q6 SF10 (60 M rows) and Q6 SF100: exact, against the
   oracle's brute-force loop run over row chunks of the host-generated table
   (aggregates decompose over row ranges, pin P8; the chunks run in parallel
   threads, each chunk a plain single-threaded oracle call).
@@ -74,8 +74,10 @@ def test_q1_sf100_exact():
     assert exp[3][3] > 2**63  # (N,O) sum_charge exceeds int64 at SF100 (reading A17)
 
 
-def test_q6_sf10_exact():
-    sf = 10.0
+@pytest.mark.parametrize("sf", [10.0, 100.0])
+def test_q6_exact(sf):
+    """C3 (Q6 SF10) and north_star's target config, Q6 at SF100 (600 M rows,
+    16.8 GB of columns), through the fragment bench.py times."""
     n = gen.lineitem_rows(sf)
     cols, views = device_columns(plans.Q6_COLS, n, sf)
     got, frag = run(plans.q6(), views, n)

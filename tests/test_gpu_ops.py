@@ -4,6 +4,8 @@ Selection positions, gathers, scatters, partitions and integer folds must be
 bit-exact; float folds agree within 1e-9 relative (BASELINE.json north_star)
 -- the oracle accumulates in long double, the GPU in f64.
 """
+import zlib
+
 import numpy as np
 import pytest
 import torch
@@ -249,7 +251,7 @@ def _run_fold(op, a, c, n, dtype_np):
 @pytest.mark.parametrize("kind", CTRLS)
 def test_fold_vs_interpreter(op, dtype, kind):
     n = 20011
-    rng = np.random.default_rng(abs(hash((op, dtype, str(kind)))) % 2**32)
+    rng = np.random.default_rng(zlib.crc32(repr((op, dtype, kind)).encode()))
     if dtype == "u8":
         a = rng.integers(0, 250, n).astype(np.uint8)
     elif dtype == "i32":
@@ -333,7 +335,7 @@ def test_fold_scan_vs_interpreter(dtype, kind, n):
     longer than a tile, irregular virtual and materialized controls.  Integer
     exact; float within 1e-9 relative of the long-double oracle (positive
     data: no cancellation)."""
-    rng = np.random.default_rng(abs(hash((dtype, str(kind), n))) % 2**32)
+    rng = np.random.default_rng(zlib.crc32(repr((dtype, kind, n)).encode()))
     if dtype == "u8":
         a = rng.integers(0, 250, n).astype(np.uint8)
     elif dtype == "i32":
