@@ -63,6 +63,7 @@ def parse():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     ap.add_argument("--seed", type=int, default=0x5EEDC0DE)
+    ap.add_argument("--no-graph", action="store_true", help="N > 1: launch eagerly instead of CUDA graphs")
     ap.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
                     help="process-group backend for N > 1 (gloo: test mode, ranks may share a GPU)")
     return ap.parse_args()
@@ -440,17 +441,53 @@ def main():
     pbytes = vd.partials_bytes(plan)
     out = torch.empty(pbytes, dtype=torch.uint8, device=dev)
     ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
-    gathered = torch.empty(pbytes * world, dtype=torch.uint8, device=dev) if world > 1 else None
+    gathered = torch.empty(pbytes * world, dtype=torch.uint8, device=dev) if world > 1 else out
+    result = vd.DeviceResult(plan, dev)
 
-    def step():
+    # A step: the fused fragment over this rank's rows (a2-a9), then the
+    # cross-GPU step (all-gather of the partials, N > 1) and the device merge
+    # + Fig 11 compaction into a vd_result -- the query's answer is on the
+    # device when the step ends (no host round trip).
+    def pipe():
         vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
+
+    def exchange():
         comm.all_gather(out, gathered)
+        vd.merge_partials_device(plan, views, dim_views, gathered, world, result, stream=stream)
 
     steps = args.steps if args.steps is not None else (300 if w in ("q1", "q19", "q9") else 1000)
     for _ in range(max(args.warmup, 0)):
-        step()
-    launches_per_step = vd.last_launch_count()
+        pipe()
+        launches_per_step = vd.last_launch_count()
+        exchange()
+        launches_per_step += vd.last_launch_count()
+    frag = vd.last_fragment()
     torch.cuda.synchronize()
+    # N > 1: the two halves of the step replayed as CUDA graphs (launch
+    # latency off the critical path of ~0.4 ms shards); N = 1 runs eagerly
+    graphs = None
+    if world > 1 and comm.backend == "nccl" and not args.no_graph:
+        try:
+            g1, g2 = torch.cuda.CUDAGraph(), torch.cuda.CUDAGraph()
+            side = torch.cuda.Stream(device=dev)
+            side.wait_stream(stream)
+            with torch.cuda.stream(side):
+                with torch.cuda.graph(g1, stream=side):
+                    vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=side)
+                with torch.cuda.graph(g2, stream=side):
+                    comm.all_gather(out, gathered)
+                    vd.merge_partials_device(plan, views, dim_views, gathered, world, result, stream=side)
+            stream.wait_stream(side)
+            torch.cuda.synchronize()
+            graphs = (g1, g2)
+            pipe = g1.replay  # noqa: F811
+            exchange = g2.replay  # noqa: F811
+            for _ in range(2):
+                pipe()
+                exchange()
+            torch.cuda.synchronize()
+        except Exception as e:  # capture unsupported here: stay eager, say so
+            graphs = f"eager (capture failed: {type(e).__name__}: {e})"[:200]
 
     # ---- timed region --------------------------------------------------------
     clocks = ClockSampler(local)
@@ -465,9 +502,9 @@ def main():
     t_start.record(stream)
     for i in range(steps):
         ev[i][0].record(stream)
-        vd.run_pipeline(plan, views, n, dim_views, out=out, ws=ws, stream=stream)
+        pipe()
         ev[i][1].record(stream)
-        comm.all_gather(out, gathered)
+        exchange()
     t_end.record(stream)
     torch.cuda.synchronize()
     comm.barrier()
@@ -478,14 +515,13 @@ def main():
     elapsed_ms, kernel_ms = comm.max([elapsed_ms, kernel_ms])
     ms_per_step = elapsed_ms / steps
 
-    # result check (merge of the per-rank partials, host side)
-    if world > 1:
-        parts = [gathered[r * pbytes:(r + 1) * pbytes].cpu().numpy().tobytes() for r in range(world)]
-        merged = vd.merge_partials(plan, views, dim_views, parts)
-    else:
-        merged = out.cpu().numpy().tobytes()
+    # the step's answer: the device vd_result (merged + compacted on the GPU)
     fl = [w == "select"] + [False] * 8
-    result = vd.decode_partials(merged, plan, float_aggs=fl)
+    result_dev = result
+    result = result_dev.decode(plan, float_aggs=fl)
+    if world > 1:  # cross-check against the host merge of the gathered partials
+        parts = [gathered[r * pbytes:(r + 1) * pbytes].cpu().numpy().tobytes() for r in range(world)]
+        assert vd.merge_partials(plan, views, dim_views, parts, float_aggs=fl) == result
 
     # ---- e2e: host buffers in, result out, through the public API -------------
     e2e = None
@@ -505,7 +541,7 @@ def main():
         looked_up = n if args.sel_mode == "predicated" else sel_rows // max(world, 1)
         alg_bytes = n * bpr + 64 * looked_up
         extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64}
-        if vd.last_fragment() == "late":
+        if frag == "late":
             # late materialisation (A31/A33/A34): fact.v in full, of fact.fk
             # the 64-byte blocks holding a qualifying row, 64 B per lookup
             thr = int(round(args.selectivity * plans.FKJSEL_VMAX))
@@ -518,7 +554,7 @@ def main():
             extra = {"bytes_per_row_dense": bpr, "lookups": looked_up, "lookup_granule_bytes": 64,
                      "fk_blocks": fk_blocks}
             del mask
-    elif w == "q19" and vd.last_fragment() == "late":
+    elif w == "q19" and frag == "late":
         # late-materialisation fragment, readings A31/A33: the lead columns
         # (l_shipmode, l_shipinstruct: the u8 terms every conjunction shares)
         # in full; of l_partkey / l_quantity the 64-byte blocks holding a
@@ -555,7 +591,8 @@ def main():
         "dtype": "f32/f64" if w == "select" else "int64",
         "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
         "config": bench_config(args, w, sf, world),
-        "fragment": "generic" if args.generic else vd.last_fragment(),
+        "fragment": "generic" if args.generic else frag,
+        "cuda_graphs": ("pipeline + (all-gather, merge)" if isinstance(graphs, tuple) else graphs),
         "hbm_gbs": achieved,
         "roofline": hbm_roofline(
             achieved, "k_pipe_q1_tma" if w == "q1" and not args.generic else "vd_run_pipeline", kernel_ms,
@@ -1108,7 +1145,10 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
         h.copy_(c)
     dst = [torch.empty_like(c) for c in cols]
     out = torch.empty(pbytes, dtype=torch.uint8, device=dev)
-    res = torch.empty(pbytes, dtype=torch.uint8, pin_memory=pinned)
+    gathered = torch.empty(pbytes * world, dtype=torch.uint8, device=dev) if world > 1 else out
+    result = vd.DeviceResult(plan, dev)
+    rbufs = [result.ngroups, result.keys, result.rows, result.aggs]
+    hres = [torch.empty(t.numel(), dtype=t.dtype, pin_memory=pinned) for t in rbufs]
     ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plan), dev)
     reps = 3
     torch.cuda.synchronize()
@@ -1121,13 +1161,17 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
             c.min, c.max, c.has_minmax, c.flags = v.min, v.max, v.has_minmax, v.flags  # catalog metadata
             vcols.append(c)
         vd.run_pipeline(plan, vcols, n, dim_views, out=out, ws=ws, stream=stream)
-        res.copy_(out, non_blocking=True)
+        comm.all_gather(out, gathered)
+        vd.merge_partials_device(plan, vcols, dim_views, gathered, world, result, stream=stream)
+        for h, d in zip(hres, rbufs):  # the compacted result back to the host
+            h.copy_(d, non_blocking=True)
         torch.cuda.synchronize()
     dt = (time.perf_counter() - t0) / reps
     dt = comm.max([dt])[0]
     h2d = sum(c.numel() * c.element_size() for c in cols)
+    d2h = sum(t.numel() * t.element_size() for t in rbufs)
     del host, dst
-    return {"value": (n * world) / dt, "unit": "rows/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": pbytes,
+    return {"value": (n * world) / dt, "unit": "rows/s", "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h,
             "pinned": pinned, "reps": reps, "s_per_step": dt}
 
 

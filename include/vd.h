@@ -424,23 +424,57 @@ vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const v
                         const vd_agg* aggs, int32_t naggs, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
                         int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
 
-/* Host merge of per-device partials (rank order, exact 128-bit / f64), the
- * cross-GPU step of the hierarchical fold (Fig 3 one level up):
- * parts_host[r] points to rank r's partials copied to the host.  out_host
- * receives one merged partials buffer (same layout).  cols / dims are the
- * column views the plan was run with (only dtypes are read: they decide
- * which aggregates are f64). */
+/* Compacted result of a pipeline: the FoldSelect compaction of Fig 11
+ * applied to the merged partials -- the non-empty groups
+ * (row count > 0), in ascending key order (reading A16), empty groups
+ * dropped.  Every pointer is caller-owned; HOST memory for
+ * vd_merge_partials, DEVICE memory for vd_merge_partials_device.
+ *   keys    : int64 [capacity], the group key (index in [0, plan->ngroups))
+ *   aggs    : [capacity][plan->naggs] 16-byte slots, encoded as in
+ *             vd_partials (integer SUM/COUNT int128; float SUM f64 in the
+ *             low 8 bytes; MIN/MAX int64 / f64 in the low 8 bytes)
+ *   rows    : int64 [capacity], the group's row count (> 0)
+ *   ngroups : int64 scalar, the number of groups written
+ * capacity >= plan->ngroups (else VD_E_SHAPE). */
+typedef struct {
+    int64_t capacity;
+    int64_t* keys;
+    void* aggs;
+    int64_t* rows;
+    int64_t* ngroups;
+} vd_result;
+
+/* Merge of per-device partials, the cross-GPU step of the hierarchical fold
+ * (Fig 3 one level up), followed by the Fig 11 compaction:
+ * parts_host[r] points to rank r's vd_partials copied to the host; they are
+ * combined in rank order (SUM/COUNT exact in 128 bits or f64; MIN/MAX over
+ * the ranks where the group is non-empty) and the non-empty groups are
+ * written to *out (host buffers).  cols / dims are the column views the plan
+ * ran with: only their dtypes are read (they decide which aggregates are
+ * f64); they may be NULL when nparts == 1 (a single partial is compacted,
+ * nothing is added). */
 vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int32_t ncols, const vd_column* dims,
-                            int32_t ndims, const void* const* parts_host, int32_t nparts, void* out_host);
+                            int32_t ndims, const void* const* parts_host, int32_t nparts, const vd_result* out);
+
+/* The same merge + compaction on the device, in one kernel (one CTA) on
+ * `stream`: parts_dev holds nparts vd_partials buffers back to back (e.g.
+ * the output of an all-gather of every rank's partials, rank order), and
+ * *out's buffers are device memory.  For nparts == 1 it is the device-side
+ * finalisation of a single GPU's pipeline.  Stream-ordered: nothing is
+ * synchronised; *out->ngroups is valid once the stream reaches the kernel's
+ * end.  cols/dims as vd_merge_partials. */
+vd_status vd_merge_partials_device(const vd_pipeline* plan, const vd_column* cols, int32_t ncols,
+                                   const vd_column* dims, int32_t ndims, const void* parts_dev, int32_t nparts,
+                                   const vd_result* out, void* stream);
 
 /* Rows whose group key fell outside [0, ngroups) in the last generic-path
  * vd_run_pipeline on `ws` (device int64 at ws + 128; read after the stream
  * synchronises).  They are dropped, not folded. */
 #define VD_WS_DOMAIN_ERRORS_OFFSET 128
 
-/* sizeof() of the ABI structs, for binding self-checks: out[0..7] =
+/* sizeof() of the ABI structs, for binding self-checks: out[0..8] =
  * vd_column, vd_ctrl, vd_term, vd_conj, vd_pred, vd_agg, vd_keypart,
- * vd_pipeline.  Returns the number written (<= n). */
+ * vd_pipeline, vd_result.  Returns the number written (<= n). */
 int32_t vd_abi_struct_sizes(size_t* out, int32_t n);
 
 /* Name of the fragment the last vd_run_pipeline on this thread ran:

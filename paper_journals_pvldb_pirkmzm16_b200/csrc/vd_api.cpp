@@ -285,10 +285,11 @@ int32_t vd_last_launch_count(void) { return t_launches; }
 const char* vd_last_fragment(void) { return t_fragment; }
 
 int32_t vd_abi_struct_sizes(size_t* out, int32_t n) {
-    const size_t v[8] = {sizeof(vd_column), sizeof(vd_ctrl), sizeof(vd_term), sizeof(vd_conj),
-                         sizeof(vd_pred), sizeof(vd_agg), sizeof(vd_keypart), sizeof(vd_pipeline)};
+    const size_t v[9] = {sizeof(vd_column), sizeof(vd_ctrl),     sizeof(vd_term),
+                         sizeof(vd_conj),   sizeof(vd_pred),     sizeof(vd_agg),
+                         sizeof(vd_keypart), sizeof(vd_pipeline), sizeof(vd_result)};
     int32_t k = 0;
-    for (; k < n && k < 8; ++k) out[k] = v[k];
+    for (; k < n && k < 9; ++k) out[k] = v[k];
     return k;
 }
 
@@ -729,21 +730,47 @@ vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const v
     return st;
 }
 
-vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int32_t ncols, const vd_column* dims,
-                            int32_t ndims, const void* const* parts, int32_t nparts, void* out_host) {
-    if (!plan || !out_host || (nparts > 0 && !parts)) return VD_E_NULL;
-    if (plan->ngroups < 1 || plan->naggs < 0 || plan->naggs > VD_MAX_AGGS) return VD_E_ARG;
-    const int NA = plan->naggs;
-    const int64_t G = plan->ngroups;
-    bool isf[VD_MAX_AGGS] = {false};
-    for (int a = 0; a < NA; ++a) {
+// Which aggregates of `plan` are f64 (a float factor column); cols/dims may
+// be NULL (then every aggregate reads as integer: only valid for nparts == 1,
+// where nothing is added).
+static vd_status merge_prologue(const vd_pipeline* plan, const vd_column* cols, int32_t ncols,
+                                const vd_column* dims, int32_t ndims, int32_t nparts, const vd_result* out,
+                                int32_t* isf) {
+    if (!plan || !out || !out->keys || !out->rows || !out->ngroups || (plan->naggs > 0 && !out->aggs))
+        return VD_E_NULL;
+    if (plan->ngroups < 1 || plan->ngroups > VD_MAX_GROUPS || plan->naggs < 0 || plan->naggs > VD_MAX_AGGS)
+        return VD_E_ARG;
+    if (nparts < 1) { set_error("merge: nparts < 1"); return VD_E_SHAPE; }
+    if (out->capacity < plan->ngroups) { set_error("vd_result capacity < plan->ngroups"); return VD_E_SHAPE; }
+    if (nparts > 1 && !cols && !dims) {  // the dtypes decide int128 vs f64 addition
+        for (int a = 0; a < plan->naggs; ++a)
+            if (plan->aggs[a].kind != VD_AGG_COUNT && plan->aggs[a].nfactors > 0) {
+                set_error("merge of several partials needs the column views (their dtypes)");
+                return VD_E_NULL;
+            }
+    }
+    for (int a = 0; a < VD_MAX_AGGS; ++a) isf[a] = 0;
+    for (int a = 0; a < plan->naggs; ++a) {
         const vd_agg& g = plan->aggs[a];
-        if (g.kind == VD_AGG_COUNT) continue;
+        if (g.kind == VD_AGG_COUNT || (!cols && !dims)) continue;
         for (int f = 0; f < g.nfactors; ++f) {
             int dt = plan_col_dtype(plan, cols, ncols, dims, ndims, g.f[f].col);
-            if (dt == VD_F32 || dt == VD_F64) isf[a] = true;
+            if (dt == VD_F32 || dt == VD_F64) isf[a] = 1;
         }
     }
+    return VD_OK;
+}
+
+vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int32_t ncols, const vd_column* dims,
+                            int32_t ndims, const void* const* parts, int32_t nparts, const vd_result* out) {
+    int32_t isf[VD_MAX_AGGS];
+    vd_status st = merge_prologue(plan, cols, ncols, dims, ndims, nparts, out, isf);
+    if (st != VD_OK) return st;
+    if (!parts) return VD_E_NULL;
+    for (int r = 0; r < nparts; ++r)
+        if (!parts[r]) return VD_E_NULL;
+    const int NA = plan->naggs;
+    const int64_t G = plan->ngroups;
     typedef __int128 I;
     auto rd = [](const void* p, int64_t k) {
         const uint64_t* q = (const uint64_t*)p + 2 * k;
@@ -754,11 +781,13 @@ vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int3
         std::memcpy(&d, (const uint64_t*)p + 2 * k, 8);
         return d;
     };
-    uint64_t* o = (uint64_t*)out_host;
-    for (int64_t g = 0; g < G; ++g) {
+    uint64_t* oa = (uint64_t*)out->aggs;
+    int64_t ng = 0;
+    for (int64_t g = 0; g < G; ++g) {  // ascending key: the pivot order of Fig 11
         const int64_t base = g * (NA + 1);
         I rows = 0;
         for (int r = 0; r < nparts; ++r) rows += rd(parts[r], base + NA);
+        if (rows == 0) continue;  // empty group: dropped by the compaction (A16)
         for (int a = 0; a < NA; ++a) {
             const int kind = plan->aggs[a].kind;
             I vi = 0;
@@ -778,8 +807,10 @@ vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int3
                 }
                 have = true;
             }
-            uint64_t* q = o + 2 * (base + a);
-            if (isf[a] && kind != VD_AGG_COUNT) {
+            uint64_t* q = oa + 2 * (ng * NA + a);
+            if (nparts == 1) {  // a single partial: the slot verbatim
+                std::memcpy(q, (const uint64_t*)parts[0] + 2 * (base + a), 16);
+            } else if (isf[a] && kind != VD_AGG_COUNT) {
                 std::memcpy(q, &vf, 8);
                 q[1] = 0;
             } else {
@@ -787,10 +818,26 @@ vd_status vd_merge_partials(const vd_pipeline* plan, const vd_column* cols, int3
                 q[1] = (uint64_t)((unsigned __int128)vi >> 64);
             }
         }
-        uint64_t* q = o + 2 * (base + NA);
-        q[0] = (uint64_t)(unsigned __int128)rows;
-        q[1] = (uint64_t)((unsigned __int128)rows >> 64);
+        out->keys[ng] = g;
+        out->rows[ng] = (int64_t)rows;
+        ++ng;
     }
+    *out->ngroups = ng;
+    return VD_OK;
+}
+
+vd_status vd_merge_partials_device(const vd_pipeline* plan, const vd_column* cols, int32_t ncols,
+                                   const vd_column* dims, int32_t ndims, const void* parts_dev, int32_t nparts,
+                                   const vd_result* out, void* stream) {
+    reset_launches();
+    int32_t isf[VD_MAX_AGGS];
+    vd_status st = merge_prologue(plan, cols, ncols, dims, ndims, nparts, out, isf);
+    if (st != VD_OK) return st;
+    if (!parts_dev) return VD_E_NULL;
+    int nl = 0;
+    cudaError_t e = launch_merge_partials(plan, isf, parts_dev, nparts, *out, (cudaStream_t)stream, &nl);
+    count_launches(nl);
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     return VD_OK;
 }
 

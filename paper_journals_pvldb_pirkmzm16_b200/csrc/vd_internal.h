@@ -107,6 +107,10 @@ cudaError_t launch_group_fold(const DevCols& cols, const DevPred& pred, int64_t 
                               void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws, cudaStream_t s,
                               int* nl);
 
+// k_merge.cu: rank-order merge of nparts device partials + Fig 11 compaction
+cudaError_t launch_merge_partials(const vd_pipeline* plan, const int32_t* isf, const void* parts, int nparts,
+                                  const vd_result& out, cudaStream_t s, int* nl);
+
 int num_sms();
 
 }  // namespace vd

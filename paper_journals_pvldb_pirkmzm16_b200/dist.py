@@ -49,11 +49,35 @@ def all_gather_partials(local, group=None) -> List[bytes]:
 
 
 def merge(plan: vd.vd_pipeline, cols: Sequence[vd.vd_column], dims: Sequence[vd.vd_column],
-          parts: Sequence[bytes]) -> bytes:
-    """Rank-order merge of per-rank partials (vd_merge_partials, host)."""
-    return vd.merge_partials(plan, cols, dims, parts)
+          parts: Sequence[bytes], float_aggs: Sequence[bool] = ()):
+    """Rank-order merge of per-rank partials + the Fig 11 compaction
+    (vd_merge_partials, host): {group: [aggs..., rows]}."""
+    return vd.merge_partials(plan, cols, dims, parts, float_aggs)
 
 
-def exchange_and_merge(plan, cols, dims, local, group=None) -> bytes:
-    """The cross-GPU step of the hierarchical fold: all-gather + merge."""
-    return merge(plan, cols, dims, all_gather_partials(local, group))
+def exchange_and_merge(plan, cols, dims, local, group=None, float_aggs: Sequence[bool] = ()):
+    """The cross-GPU step of the hierarchical fold: all-gather + host merge."""
+    return merge(plan, cols, dims, all_gather_partials(local, group), float_aggs)
+
+
+class DeviceExchange:
+    """The cross-GPU step kept on the device (no host round trip): NCCL
+    all_gather_into_tensor of every rank's partials into one buffer, then
+    vd_merge_partials_device (one CTA: rank-order int128/f64 merge + Fig 11
+    compaction) into a device vd_result -- both enqueued on the caller's
+    stream, so the pair can be captured in a CUDA graph behind the pipeline
+    launch.  world == 1 skips the collective (the merge is the compaction)."""
+
+    def __init__(self, plan, cols, dims, local, world: int, group=None):
+        import torch
+        self.plan, self.cols, self.dims, self.local, self.world, self.group = plan, cols, dims, local, world, group
+        nb = local.numel()
+        self.gathered = (torch.empty(nb * world, dtype=torch.uint8, device=local.device) if world > 1 else local)
+        self.result = vd.DeviceResult(plan, local.device)
+
+    def step(self, stream=None):
+        if self.world > 1:
+            import torch.distributed as dist
+            dist.all_gather_into_tensor(self.gathered, self.local, group=self.group)
+        vd.merge_partials_device(self.plan, self.cols, self.dims, self.gathered, self.world, self.result, stream)
+        return self.result

@@ -91,6 +91,11 @@ class vd_pipeline(Structure):
                 ("force_generic", c_int32), ("aggs", vd_agg * VD_MAX_AGGS)]
 
 
+class vd_result(Structure):
+    _fields_ = [("capacity", c_int64), ("keys", c_void_p), ("aggs", c_void_p), ("rows", c_void_p),
+                ("ngroups", c_void_p)]
+
+
 _P = POINTER
 _sigs = {
     "vd_status_str": (ctypes.c_char_p, [c_int32]),
@@ -126,7 +131,9 @@ _sigs = {
     "vd_run_pipeline": (c_int32, [_P(vd_pipeline), _P(vd_column), c_int32, c_int64, _P(vd_column), c_int32,
                                   c_void_p, c_void_p, c_size_t, c_void_p]),
     "vd_merge_partials": (c_int32, [_P(vd_pipeline), _P(vd_column), c_int32, _P(vd_column), c_int32,
-                                    _P(c_void_p), c_int32, c_void_p]),
+                                    _P(c_void_p), c_int32, _P(vd_result)]),
+    "vd_merge_partials_device": (c_int32, [_P(vd_pipeline), _P(vd_column), c_int32, _P(vd_column), c_int32,
+                                           c_void_p, c_int32, _P(vd_result), c_void_p]),
     "vd_group_fold_ws_bytes": (c_int32, [c_int64, c_int32, _P(c_size_t)]),
     "vd_group_fold": (c_int32, [_P(vd_column), c_int32, c_int64, _P(vd_pred), c_int32, _P(vd_agg), c_int32,
                                 c_void_p, c_void_p, c_void_p, c_void_p, c_void_p, c_size_t, c_void_p]),
@@ -142,10 +149,10 @@ for _name, (_res, _args) in _sigs.items():
 
 
 def _check_abi():
-    out = (c_size_t * 8)()
-    _L.vd_abi_struct_sizes(out, 8)
+    out = (c_size_t * 9)()
+    _L.vd_abi_struct_sizes(out, 9)
     mine = [ctypes.sizeof(t) for t in (vd_column, vd_ctrl, vd_term, vd_conj, vd_pred, vd_agg, vd_keypart,
-                                       vd_pipeline)]
+                                       vd_pipeline, vd_result)]
     if list(out) != mine:
         raise ImportError(f"libvd ABI struct sizes {list(out)} != binding {mine}")
 
@@ -227,6 +234,18 @@ def column(t, minmax: Optional[Sequence[int]] = None, scale: int = 0, length: Op
     if noeps:
         c.flags |= VD_COL_NOEPS
     c._keep = t  # the view keeps its tensor alive (the ABI struct holds a raw pointer)
+    return c
+
+
+def column_meta(dtype) -> vd_column:
+    """A vd_column carrying only a dtype (vd_dtype int or numpy dtype), no
+    data: what vd_merge_partials reads of the views a plan ran with."""
+    import numpy as np
+    c = vd_column()
+    if not isinstance(dtype, int):
+        dtype = {np.dtype(np.uint8): VD_U8, np.dtype(np.int32): VD_I32, np.dtype(np.int64): VD_I64,
+                 np.dtype(np.float32): VD_F32, np.dtype(np.float64): VD_F64}[np.dtype(dtype)]
+    c.dtype = dtype
     return c
 
 
@@ -550,37 +569,102 @@ def run_pipeline(plan: vd_pipeline, cols: Sequence[vd_column], n: int, dims: Seq
                            out.data_ptr(), ws.data_ptr(), ws.numel(), _stream(stream)), "vd_run_pipeline")
 
 
-def merge_partials(plan: vd_pipeline, cols: Sequence[vd_column], dims: Sequence[vd_column], parts_host) -> bytes:
-    """vd_merge_partials over host byte buffers (rank order); returns the merged buffer."""
+class HostResult:
+    """Host buffers of a vd_result (capacity = plan.ngroups groups)."""
+
+    def __init__(self, plan: vd_pipeline):
+        cap = int(plan.ngroups)
+        self.naggs = int(plan.naggs)
+        self.keys = (ctypes.c_int64 * cap)()
+        self.aggs = ctypes.create_string_buffer(max(1, cap * self.naggs * 16))
+        self.rows = (ctypes.c_int64 * cap)()
+        self.ngroups = ctypes.c_int64(0)
+        self.struct = vd_result(cap, ctypes.addressof(self.keys), ctypes.addressof(self.aggs),
+                                ctypes.addressof(self.rows), ctypes.addressof(self.ngroups))
+
+    def decode(self, plan: vd_pipeline, float_aggs: Sequence[bool] = ()):
+        g = int(self.ngroups.value)
+        return decode_result(bytes(self.keys)[:8 * g], self.aggs.raw[:16 * g * self.naggs], bytes(self.rows)[:8 * g],
+                             g, plan, float_aggs)
+
+
+class DeviceResult:
+    """Device buffers of a vd_result (torch CUDA tensors)."""
+
+    def __init__(self, plan: vd_pipeline, device=None):
+        torch = _torch()
+        cap = int(plan.ngroups)
+        self.naggs = int(plan.naggs)
+        self.keys = torch.empty(cap, dtype=torch.int64, device=device or "cuda")
+        self.aggs = torch.empty(max(1, cap * self.naggs * 16), dtype=torch.uint8, device=self.keys.device)
+        self.rows = torch.empty(cap, dtype=torch.int64, device=self.keys.device)
+        self.ngroups = torch.zeros(1, dtype=torch.int64, device=self.keys.device)
+        self.struct = vd_result(cap, self.keys.data_ptr(), self.aggs.data_ptr(), self.rows.data_ptr(),
+                                self.ngroups.data_ptr())
+
+    def decode(self, plan: vd_pipeline, float_aggs: Sequence[bool] = ()):
+        """Copy the written groups to the host and decode them (synchronises)."""
+        g = int(self.ngroups.item())
+        return decode_result(self.keys[:g].cpu().numpy().tobytes(),
+                             self.aggs[:16 * g * self.naggs].cpu().numpy().tobytes(),
+                             self.rows[:g].cpu().numpy().tobytes(), g, plan, float_aggs)
+
+
+def merge_partials(plan: vd_pipeline, cols: Sequence[vd_column], dims: Sequence[vd_column], parts_host,
+                   float_aggs: Sequence[bool] = ()):
+    """vd_merge_partials over host byte buffers (rank order): the merged,
+    compacted result decoded as {group: [agg values..., row_count]}."""
     nb = partials_bytes(plan)
     bufs = [ctypes.create_string_buffer(bytes(b), nb) for b in parts_host]
     ptrs = (c_void_p * max(1, len(bufs)))(*[ctypes.addressof(b) for b in bufs])
-    out = ctypes.create_string_buffer(nb)
-    _ok(_L.vd_merge_partials(ctypes.byref(plan), _cols_array(cols), len(cols), _cols_array(dims), len(dims), ptrs,
-                             len(bufs), out), "vd_merge_partials")
-    return out.raw
+    res = HostResult(plan)
+    _ok(_L.vd_merge_partials(ctypes.byref(plan), _cols_array(cols) if cols else None, len(cols),
+                             _cols_array(dims) if dims else None, len(dims), ptrs, len(bufs), ctypes.byref(res.struct)),
+        "vd_merge_partials")
+    return res.decode(plan, float_aggs)
+
+
+def merge_partials_device(plan: vd_pipeline, cols: Sequence[vd_column], dims: Sequence[vd_column], parts_dev,
+                          nparts: int, result: Optional[DeviceResult] = None, stream=None) -> DeviceResult:
+    """vd_merge_partials_device: rank-order merge of `nparts` partials held
+    back to back in the CUDA tensor `parts_dev`, compacted into `result`
+    (allocated if None) on `stream`; nothing synchronises."""
+    if result is None:
+        result = DeviceResult(plan, parts_dev.device)
+    _ok(_L.vd_merge_partials_device(ctypes.byref(plan), _cols_array(cols) if cols else None, len(cols),
+                                    _cols_array(dims) if dims else None, len(dims), parts_dev.data_ptr(), nparts,
+                                    ctypes.byref(result.struct), _stream(stream)), "vd_merge_partials_device")
+    return result
+
+
+def decode_result(keys: bytes, aggs: bytes, rows: bytes, ngroups: int, plan: vd_pipeline,
+                  float_aggs: Sequence[bool] = ()):
+    """Byte decoding of a vd_result's first `ngroups` groups (no filtering,
+    no arithmetic: the library did the compaction): {key: [agg values...,
+    row_count]} in the library's order; integer slots as exact Python ints,
+    slots flagged in float_aggs as f64."""
+    import struct
+    na = int(plan.naggs)
+    res = {}
+    for j in range(ngroups):
+        (k,) = struct.unpack_from("<q", keys, 8 * j)
+        (r,) = struct.unpack_from("<q", rows, 8 * j)
+        vals = []
+        for a in range(na):
+            off = (j * na + a) * 16
+            if a < len(float_aggs) and float_aggs[a] and plan.aggs[a].kind != VD_AGG_COUNT:
+                vals.append(struct.unpack_from("<d", aggs, off)[0])
+            else:
+                lo, hi = struct.unpack_from("<Qq", aggs, off)
+                vals.append(hi * (1 << 64) + lo)
+        vals.append(r)
+        res[k] = vals
+    return res
 
 
 def decode_partials(buf: bytes, plan: vd_pipeline, float_aggs: Sequence[bool] = ()):
-    """{group: [agg values..., row_count]} for non-empty groups (the FoldSelect
-    compaction of Fig 11: empty groups dropped, ascending key)."""
-    import struct
-    na = plan.naggs
-    res = {}
-    for g in range(plan.ngroups):
-        base = g * (na + 1) * 16
-        lo, hi = struct.unpack_from("<Qq", buf, base + na * 16)
-        rows = hi * (1 << 64) + lo
-        if rows == 0:
-            continue
-        vals = []
-        for a in range(na):
-            off = base + a * 16
-            if a < len(float_aggs) and float_aggs[a] and plan.aggs[a].kind != VD_AGG_COUNT:
-                vals.append(struct.unpack_from("<d", buf, off)[0])
-            else:
-                lo, hi = struct.unpack_from("<Qq", buf, off)
-                vals.append(hi * (1 << 64) + lo)
-        vals.append(rows)
-        res[g] = vals
-    return res
+    """{group: [agg values..., row_count]} of ONE device's partials (copied
+    to the host): the library's vd_merge_partials with nparts = 1 does the
+    Fig 11 compaction (empty groups dropped, ascending key); this function
+    only decodes the bytes."""
+    return merge_partials(plan, [], [], [buf], float_aggs)

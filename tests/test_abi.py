@@ -24,7 +24,7 @@ def test_header_declares_the_north_star_calls():
     names = declared_functions()
     for want in ["vd_load_column", "vd_select_branch", "vd_select_predicated", "vd_gather", "vd_scatter",
                  "vd_fold_sum", "vd_fold_count", "vd_fold_min", "vd_fold_max", "vd_fold_select", "vd_run_pipeline",
-                 "vd_merge_partials", "vd_workspace_bytes", "vd_partition"]:
+                 "vd_merge_partials", "vd_merge_partials_device", "vd_workspace_bytes", "vd_partition"]:
         assert want in names
 
 
@@ -135,9 +135,41 @@ def test_merge_partials_rank_order_int128_and_empty_groups():
     big = 2**63 - 1
     r0 = _pack([big, 5, 9, 2, 2] + [0, 0, 0, 0, 0] + [7, -3, -3, 1, 1])
     r1 = _pack([big, 1, 4, 3, 3] + [0, 0, 0, 0, 0] + [0, 0, 0, 0, 0])
-    merged = vd.merge_partials(plan, [c0, c1], [], [r0, r1])
-    res = vd.decode_partials(merged, plan)
+    res = vd.merge_partials(plan, [c0, c1], [], [r0, r1])
     assert res == {0: [2 * big, 1, 9, 5, 5], 2: [7, -3, -3, 1, 1]}
+    assert list(res) == [0, 2]  # ascending key, the empty group 1 dropped (Fig 11, A16)
+    # the dtypes decide int128 vs f64 addition: several partials need the views
+    with pytest.raises(vd.VdError):
+        vd.merge_partials(plan, [], [], [r0, r1])
+
+
+def test_merge_partials_float_sum_and_single_partial_compaction():
+    """f64 SUM slots add as doubles; one partial is compacted verbatim
+    (decode_partials = vd_merge_partials with nparts = 1)."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    plan = vd.pipeline(key=[(0, 0, 0, 1)], ngroups=4, aggs=[("sum", [1]), ("count",)])
+    c0 = vd.vd_column()
+    c0.dtype = vd.VD_U8
+    c1 = vd.vd_column()
+    c1.dtype = vd.VD_F64
+    r0 = _pack([0.25, 1, 1] + [0, 0, 0] + [0, 0, 0] + [1.5, 2, 2])
+    r1 = _pack([0, 0, 0] + [0, 0, 0] + [2.0, 3, 3] + [0.125, 1, 1])
+    assert vd.merge_partials(plan, [c0, c1], [], [r0, r1], float_aggs=[True]) == \
+        {0: [0.25, 1, 1], 2: [2.0, 3, 3], 3: [1.625, 3, 3]}
+    assert vd.decode_partials(r1, plan, float_aggs=[True]) == {2: [2.0, 3, 3], 3: [0.125, 1, 1]}
+
+
+def test_binding_decodes_without_filtering():
+    """The binding only decodes what the library's vd_result holds: a
+    vd_result whose groups are written out of order and include a zero-row
+    entry comes back exactly as written (no filtering, no sorting)."""
+    import struct
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    plan = vd.pipeline(key=[(0, 0, 0, 1)], ngroups=4, aggs=[("count",)])
+    keys = struct.pack("<qqq", 3, 0, 2)
+    aggs = _pack([5, 0, 9])
+    rows = struct.pack("<qqq", 5, 0, 9)
+    assert list(vd.decode_result(keys, aggs, rows, 3, plan).items()) == [(3, [5, 5]), (0, [0, 0]), (2, [9, 9])]
 
 
 def test_pipeline_descriptor_round_trip():

@@ -2,7 +2,8 @@
 
 Each rank takes its row range (dist.shard_range), produces its partials in
 the vd_partials layout, and the ranks exchange and merge them
-(dist.exchange_and_merge: all-gather + vd_merge_partials).  With no GPU on
+(dist.exchange_and_merge: all-gather + vd_merge_partials, which also
+compacts: empty groups dropped, ascending key).  With no GPU on
 this machine the per-rank partials come from the oracle's brute-force Q1 on
 the rank's shard (packed into the ABI layout); the merged result must equal
 the whole-table oracle (pin P8)."""
@@ -52,10 +53,12 @@ def _worker(rank, world, port, ret):
     a, b = vdist.shard_range(n, rank, world, align=16)
     li = {k: gen.host(c, b - a, a, sf=sf) for k, c in gen.LINEITEM_COLS.items()}
     local = torch.frombuffer(bytearray(pack_q1(oracle.q1(li))), dtype=torch.uint8)
-    plan = plans.q1()
-    merged = vdist.exchange_and_merge(plan, [], [], local)
     from paper_journals_pvldb_pirkmzm16_b200 import vd
-    ret[rank] = {k: v[:6] for k, v in vd.decode_partials(merged, plan).items()}
+    plan = plans.q1()
+    # the merge reads only the columns' dtypes (int128 vs f64 addition)
+    views = [vd.column_meta(gen.dtype_of(gen.LINEITEM_COLS[c])) for c in plans.Q1_COLS]
+    merged = vdist.exchange_and_merge(plan, views, [], local)
+    ret[rank] = {k: v[:6] for k, v in merged.items()}
     dist.destroy_process_group()
 
 
