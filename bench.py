@@ -196,9 +196,11 @@ def host_info():
 
 
 def oracle_task(workload, sf, seed, sel_t):
-    """(make(row0, m) -> inputs, run(inputs) -> partial, merge(a, b), what):
-    the oracle program of each workload over one row range.  Partials
-    decompose over row ranges (pin P8), so a partitioned run merges them."""
+    """(make(row0, m) -> inputs, run(inputs) -> handle, extract(handle) ->
+    partial, merge(a, b), what): the oracle program of each workload over one
+    row range.  Only `run` is timed (extracting results into Python objects
+    is not the oracle's work).  Partials decompose over row ranges (pin P8),
+    so a partitioned run merges them."""
     import numpy as np
 
     import gen
@@ -214,6 +216,13 @@ def oracle_task(workload, sf, seed, sel_t):
     def add_tuple(a, b):
         return tuple(x + y for x, y in zip(a, b))
 
+    def ident(x):
+        return x
+
+    def head(p, name):
+        v, e = p.get_arrays(name)
+        return v[:1][~e[:1]].tolist()[0] if v.size and not e[0] else 0
+
     if workload in ("select", "selpos"):
         def make(row0, m):
             return gen.host(gen.F32_UNIFORM, m, row0, seed=seed)
@@ -221,13 +230,15 @@ def oracle_task(workload, sf, seed, sel_t):
             def run(v):
                 p = oracle.Program()
                 p.set("input.val", v)
-                p.run(programs.SELECT_SUM.format(intent=v.size, t=float(np.float32(sel_t)).hex()))
-                return (float(p.get("totalSum")[0] or 0.0), int(p.get("count")[0] or 0))
-            return make, run, add_tuple, "literal Voodoo interpreter, SELECT_SUM program (Fig 8 shape)"
+                return p.run(programs.SELECT_SUM.format(intent=v.size, t=float(np.float32(sel_t)).hex()))
+
+            def extract(p):
+                return (float(head(p, "totalSum")), int(head(p, "count")))
+            return make, run, extract, add_tuple, "literal Voodoo interpreter, SELECT_SUM program (Fig 8 shape)"
 
         def run(v):
             return (oracle.select_f32(v, float(np.float32(sel_t)), "lt")[1],)
-        return make, run, add_tuple, "brute-force selection loop -> int32 positions (oracle/tpch_oracle.cpp)"
+        return make, run, ident, add_tuple, "brute-force selection loop -> int32 positions (oracle/tpch_oracle.cpp)"
 
     names = {"q1": plans_cols("Q1_COLS"), "q6": plans_cols("Q6_COLS"), "q15": ["l_shipdate", "l_suppkey",
              "l_extendedprice", "l_discount"]}.get(workload, list(gen.LINEITEM_COLS))
@@ -240,23 +251,28 @@ def oracle_task(workload, sf, seed, sel_t):
             p = oracle.Program()
             for k, v in li.items():
                 p.set("lineitem." + k, v)
-            p.run(programs.Q1.format(ship_max_p1=10472))
-            keys = p.get("o_key")
-            outs = [p.get(o) for o in programs.Q1_OUTPUTS]
-            return {k: [o[j] for o in outs] for j, k in enumerate(keys) if k is not None}
-        return make, run, add_dict, "literal Voodoo interpreter, Q1 program (Fig 10/11 shape)"
+            return p.run(programs.Q1.format(ship_max_p1=10472))
+
+        def extract(p):
+            keys, ke = p.get_arrays("o_key")
+            sel = ~ke
+            outs = [p.get_arrays(o)[0][sel] for o in programs.Q1_OUTPUTS]
+            return {int(k): [int(o[j]) for o in outs] for j, k in enumerate(keys[sel].tolist())}
+        return make, run, extract, add_dict, "literal Voodoo interpreter, Q1 program (Fig 10/11 shape)"
     if workload == "q6":
         def run(li):
             p = oracle.Program()
             for k, v in li.items():
                 p.set("lineitem." + k, v)
-            p.run(programs.Q6.format(intent=1 << 30, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
-            return (int(p.get("revenue")[0] or 0), int(p.get("count")[0] or 0))
-        return make, run, add_tuple, "literal Voodoo interpreter, Q6 program (Fig 8 shape)"
+            return p.run(programs.Q6.format(intent=1 << 30, d0m1=8765, d1=9131, dlom1=4, dhip1=8, qmax=2400))
+
+        def extract(p):
+            return (int(head(p, "revenue")), int(head(p, "count")))
+        return make, run, extract, add_tuple, "literal Voodoo interpreter, Q6 program (Fig 8 shape)"
     if workload == "q15":
         def run(li):
             return {k: list(v) for k, v in oracle.q15(li).items()}
-        return make, run, add_dict, "brute-force Q15 revenue-view loop (oracle/tpch_oracle.cpp)"
+        return make, run, ident, add_dict, "brute-force Q15 revenue-view loop (oracle/tpch_oracle.cpp)"
     # FK joins (C5): the brute-force join loop over the replicated dimension tables
     part = {k: gen.host(c, gen.part_rows(sf), sf=sf, seed=seed) for k, c in gen.PART_COLS.items()}
     supp = {k: gen.host(c, gen.supplier_rows(sf), sf=sf, seed=seed) for k, c in gen.SUPPLIER_COLS.items()}
@@ -264,7 +280,7 @@ def oracle_task(workload, sf, seed, sel_t):
 
     def run(li):
         return {k: list(v) for k, v in oracle.fkj(variant, li, part, supp).items()}
-    return make, run, add_dict, f"brute-force {workload.upper()}-style FK join loop (oracle/tpch_oracle.cpp)"
+    return make, run, ident, add_dict, f"brute-force {workload.upper()}-style FK join loop (oracle/tpch_oracle.cpp)"
 
 
 def plans_cols(name):
@@ -284,7 +300,7 @@ def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5, n_total=None, partitio
 
     if workload == "fkjsel":
         return None
-    make, run, merge, what = oracle_task(workload, sf, seed, sel_t)
+    make, run, extract, merge, what = oracle_task(workload, sf, seed, sel_t)
     chunk = 1 << 19
     if n_total is None:
         n_total = gen.lineitem_rows(sf) if workload not in ("select", "selpos") else 10**9
@@ -293,8 +309,10 @@ def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5, n_total=None, partitio
         m = min(chunk, n_total - row0)
         x = make(row0, m)
         t0 = time.perf_counter()
-        r = run(x)
+        h = run(x)
         t_total += time.perf_counter() - t0
+        r = extract(h)
+        del h
         res1 = r if res1 is None else merge(res1, r)
         rows_done += m
         row0 += m
@@ -306,30 +324,27 @@ def cpu_baseline(workload, sf, seed, budget_s, sel_t=0.5, n_total=None, partitio
         N = os.cpu_count() or 1
         bounds = [(i * rows_done // N, (i + 1) * rows_done // N) for i in range(N)]
         sub = 1 << 17
-        work = [[make(a0, min(sub, b0 - a0)) for a0 in range(a, b, sub)] for a, b in bounds]
+        work = [[make(a0, min(sub, b - a0)) for a0 in range(a, b, sub)] for a, b in bounds]
 
         def thread(items):  # ctypes releases the GIL inside the C oracle
-            acc = None
-            for x in items:
-                r = run(x)
-                acc = r if acc is None else merge(acc, r)
-            return acc
+            return [run(x) for x in items]
 
         t0 = time.perf_counter()
         with cf.ThreadPoolExecutor(N) as ex:
-            parts = list(ex.map(thread, work))
+            handles = list(ex.map(thread, work))
         dt = time.perf_counter() - t0
         resN = None
-        for r in parts:
-            if r is not None:
+        for hs in handles:
+            for h in hs:
+                r = extract(h)
                 resN = r if resN is None else merge(resN, r)
+        del handles, work
         same = resN == res1 if workload != "select" else (
             abs(resN[0] - res1[0]) <= 1e-9 * abs(res1[0]) and resN[1] == res1[1])
         out["partitioned"] = {"value": rows_done / dt, "unit": "rows/s", "threads": N, "seconds": dt,
                               "merged_equals_single_thread": bool(same),
                               "sample": f"the same {rows_done} rows, thread i -> rows [i*S/N, (i+1)*S/N) "
                                         f"(Fig 3 control vector), sub-chunks of {sub}, partials merged"}
-        del work
     return out
 
 

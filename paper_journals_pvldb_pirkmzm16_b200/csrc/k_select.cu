@@ -499,6 +499,224 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
     }
 }
 
+// ---- fused single-pass selection (TMA ring + decoupled look-back) -------------
+// One pass, no materialised predicate: a producer warp claims tiles of
+// SF_CW x 1024 rows IN ORDER from a global counter (every predecessor of a
+// claimed tile is claimed by a running CTA: forward progress for the
+// look-back) and streams them into an SF_STAGES-deep mbarrier ring with 1D
+// bulk copies; consumer warp w turns 1024 rows of the tile into 32 ballots
+// held in registers (bit L of ballot 4q+j <-> row q*128 + 32j + L: each
+// ballot is directly a row-ordered 32-bit word) and releases the ring slot
+// at once, so HBM keeps streaming while the warp waits for its offset.
+// Warp 0 turns the warp counts into the tile aggregate and runs the
+// decoupled look-back (Merrill & Garland's single-pass scan) over per-tile
+// status words; then every warp stages its positions in shared memory --
+// branching: qualifying lanes store at their rank; predicated: cursor
+// arithmetic, every row stored at the cursor, the cursor advancing by the
+// predicate -- and streams the ascending run out with 16-byte
+// stores.  Two CTAs per SM, so one CTA's look-back wait overlaps the
+// other's work.  Replaces the 3-launch bitmap path (flag pass, scan,
+// position pass) for single interval terms on 4-byte columns.
+constexpr int SF_CW = 8;
+constexpr int SF_THREADS = SF_CW * 32 + 32;
+constexpr int SF_STAGES = 2;
+constexpr int SF_ROWS = SF_CW * 1024;         // rows per tile
+constexpr int SF_STG = 1024 + 128 + 8;        // per-warp position stage (ints)
+
+__device__ __forceinline__ void bar_consumers() {
+    asm volatile("bar.sync 1, %0;" ::"n"(SF_CW * 32) : "memory");
+}
+
+template <int MODE, typename T>
+__global__ void __launch_bounds__(SF_THREADS, 2) k_sel_fused(const T* __restrict__ col, T lo, T hi, int64_t n,
+                                                             int64_t ntiles, int32_t* __restrict__ out,
+                                                             int64_t* __restrict__ out_count,
+                                                             uint64_t* __restrict__ status,
+                                                             unsigned long long* __restrict__ tile_ctr) {
+    constexpr uint32_t TB = SF_ROWS * sizeof(T);
+    extern __shared__ __align__(128) uint8_t smem[];
+    int32_t* stage = reinterpret_cast<int32_t*>(smem + (size_t)SF_STAGES * TB);
+    uint64_t* full = reinterpret_cast<uint64_t*>(stage + SF_CW * SF_STG);
+    uint64_t* empty = full + SF_STAGES;
+    int64_t* s_tile = reinterpret_cast<int64_t*>(empty + SF_STAGES);
+    __shared__ int s_cnt[SF_CW], s_woff[SF_CW];
+    __shared__ int64_t s_base;
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int64_t nfull = n / SF_ROWS;  // tiles loaded by TMA; the ragged last one by LDG
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < SF_STAGES; ++i) {
+            mbar_init(&full[i], 1);
+            mbar_init(&empty[i], SF_CW);
+        }
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (warp == SF_CW) {
+        // ---- producer: claim tiles in order, stream them into the ring ----
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int st = 0;
+            uint32_t ph = 0;
+            for (int64_t it = 0;; ++it) {
+                if (it >= SF_STAGES) mbar_wait(&empty[st], ph ^ 1u);
+                const int64_t tile = (int64_t)atomicAdd(tile_ctr, 1ull);
+                if (tile >= ntiles) {
+                    s_tile[st] = -1;
+                    mbar_arrive(&full[st]);
+                    break;
+                }
+                s_tile[st] = tile;
+                if (tile < nfull) {
+                    mbar_expect_tx(&full[st], TB);
+                    tma_load_1d(smem + (size_t)st * TB, col + tile * SF_ROWS, TB, &full[st], pol);
+                } else {
+                    mbar_arrive(&full[st]);  // partial tile: the consumers read it from global memory
+                }
+                if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
+            }
+        }
+        return;
+    }
+    const unsigned lt = lanemask_lt();
+    int32_t* sw = stage + warp * SF_STG;
+    int st = 0;
+    uint32_t ph = 0;
+    for (;;) {
+        mbar_wait(&full[st], ph);
+        const int64_t tile = s_tile[st];
+        if (tile < 0) break;
+        const int64_t row_w = tile * SF_ROWS + (int64_t)warp * 1024;
+        // ---- flags -> 32 row-ordered ballot words ----
+        uint32_t bw[32];
+        if (tile < nfull) {
+            const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
+#pragma unroll
+            for (int k = 0; k < 32; ++k) {
+                const T v = src[k * 32 + lane];
+                bw[k] = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN (epsilon) fails
+            }
+        } else {
+#pragma unroll
+            for (int k = 0; k < 32; ++k) {
+                const int64_t r = row_w + k * 32 + lane;
+                bool f = false;
+                if (r < n) {
+                    const T v = __ldg(col + r);
+                    f = v >= lo && v <= hi;
+                }
+                bw[k] = __ballot_sync(VD_FULL, f);
+            }
+        }
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[st]);  // slot free: only the ballots are needed from here
+        if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
+        int cnt = 0;
+#pragma unroll
+        for (int k = 0; k < 32; ++k) cnt += __popc(bw[k]);
+        // ---- tile offset: warp counts -> aggregate -> decoupled look-back ----
+        if (lane == 0) s_cnt[warp] = cnt;
+        bar_consumers();
+        if (warp == 0) {
+            const int v = lane < SF_CW ? s_cnt[lane] : 0;
+            int incl = v;
+#pragma unroll
+            for (int o = 1; o < SF_CW; o <<= 1) {
+                const int u = __shfl_up_sync(VD_FULL, incl, o);
+                if (lane >= o) incl += u;
+            }
+            if (lane < SF_CW) s_woff[lane] = incl - v;
+            const int64_t agg = __shfl_sync(VD_FULL, incl, SF_CW - 1);
+            const int64_t base = lookback_exclusive_w128(status, tile, agg, lane);
+            if (lane == 0) {
+                s_base = base;
+                if (tile == ntiles - 1) *out_count = base + agg;
+            }
+        }
+        bar_consumers();
+        const int64_t g0 = s_base + s_woff[warp];
+        // ---- positions -> stage (ascending), then 16-byte streaming stores ----
+        // stage index a + k <-> output g0 + k, a = the output's misalignment
+        // in words, so stage groups of 4 are 16-byte output groups
+        const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+        int cur = a;
+#pragma unroll
+        for (int q = 0; q < 8; ++q) {
+            const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
+            int pre = cur;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                const uint32_t w = bw[4 * q + j];
+                const int f = (w >> lane) & 1u;
+                const int r = __popc(w & lt);
+                const int32_t row = (int32_t)(row_w + q * 128 + j * 32 + lane);
+                if (MODE == 0) {
+                    if (f) sw[pre + r] = row;
+                } else {
+                    // cursor arithmetic: unconditional store; rows that do not
+                    // qualify land past the block's count and are overwritten
+                    const int sel_before = pre - cur + r;
+                    const int k = f ? pre + r : cur + cq + (j * 32 + lane - sel_before);
+                    sw[k] = row;
+                }
+                pre += __popc(w);
+            }
+            cur += cq;
+        }
+        __syncwarp();
+        const int total = cur - a;
+        const int ngr = (a + total + 3) >> 2;
+        int32_t* ob = out + g0 - a;  // 16-byte aligned
+        for (int v = lane; v < ngr; v += 32) {
+            const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
+            if (4 * v >= a && 4 * v + 4 <= a + total) {
+                __stcs(reinterpret_cast<int4*>(ob) + v, x);
+            } else {
+                const int32_t xs[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+                for (int e = 0; e < 4; ++e) {
+                    const int k = 4 * v + e;
+                    if (k >= a && k < a + total) __stcs(ob + k, xs[e]);
+                }
+            }
+        }
+        __syncwarp();
+    }
+}
+
+static size_t sel_fused_smem(size_t tsize) {
+    return (size_t)SF_STAGES * SF_ROWS * tsize + (size_t)SF_CW * SF_STG * 4 + 2 * SF_STAGES * 8 + SF_STAGES * 8;
+}
+
+// VD_SELECT_FUSED=0 keeps the bitmap path (comparison runs)
+static bool use_sel_fused() {
+    static const bool off = [] {
+        const char* e = getenv("VD_SELECT_FUSED");
+        return e && strcmp(e, "0") == 0;
+    }();
+    return !off;
+}
+
+template <int MODE, typename T>
+static cudaError_t run_select_fused(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
+                                    void* ws, cudaStream_t s, int* nl) {
+    const int64_t ntiles = (n + SF_ROWS - 1) / SF_ROWS;
+    if (ntiles == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
+    unsigned long long* ctr = (unsigned long long*)ws;
+    uint64_t* status = (uint64_t*)((char*)ws + 256);
+    cudaError_t e = cudaMemsetAsync(ws, 0, 256 + (size_t)ntiles * 8, s);
+    if (e != cudaSuccess) return e;
+    const size_t sm = sel_fused_smem(sizeof(T));
+    auto kern = k_sel_fused<MODE, T>;
+    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+    int per_sm = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SF_THREADS, sm) != cudaSuccess || per_sm < 1)
+        per_sm = 1;
+    const int grid = (int)std::min<int64_t>(ntiles, (int64_t)num_sms() * per_sm);
+    kern<<<grid, SF_THREADS, sm, s>>>(col, lo, hi, n, ntiles, out_pos, out_count, status, ctr);
+    ++*nl;
+    return cudaGetLastError();
+}
+
 // Per-row predicates (several columns, run heads): ballot j is word j.
 template <class F>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_bal(F fl, int64_t n, uint32_t* __restrict__ bits,
@@ -676,7 +894,7 @@ static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t*
 }
 
 size_t select_ws_bytes(int64_t n) {
-    int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
+    int64_t ntiles = (n + std::min(SEL_TILE, SF_ROWS) - 1) / std::min(SEL_TILE, SF_ROWS);
     size_t b = 256 + (size_t)ntiles * 8;
     size_t lb = (b + 255) & ~(size_t)255;
     size_t bm = bm_ws_bytes(n);
@@ -771,6 +989,10 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
     if (aligned) {
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+        if constexpr (sizeof(T) == 4) {
+            if (ivl && use_sel_fused() && ((uintptr_t)p & 15) == 0)
+                return run_select_fused<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+        }
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L) {
                 bool tma_done = false;

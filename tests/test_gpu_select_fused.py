@@ -1,0 +1,83 @@
+"""The fused single-pass selection kernel (k_sel_fused: TMA ring, ballot
+words in registers, decoupled look-back, staged 16-byte stores) against the
+oracle, at sizes around its 8192-row tile (full tiles by TMA, the ragged
+last tile by LDG), all-false / all-true tiles, NaN (epsilon, never
+selected: A9), int32 columns, unaligned outputs, branching and predicated
+(identical positions), and the same inputs through the bitmap
+path (VD_SELECT_FUSED=0) it replaces."""
+import numpy as np
+import pytest
+import torch
+
+import gen
+import oracle
+from paper_journals_pvldb_pirkmzm16_b200 import vd
+
+from test_gpu_pipeline import env
+
+pytestmark = pytest.mark.gpu
+
+SIZES = [1, 31, 8191, 8192, 8193, 3 * 8192 + 5, 70001, 1 << 20]
+
+
+def _select(fn, v, n, t, shift=0):
+    buf = torch.full((n + 8,), -7, dtype=torch.int32, device="cuda")
+    out = buf[shift:shift + n]
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    fn([vd.column(v)], n, vd.pred([[(0, "<", t)]]), out_pos=out, out_count=cnt)
+    c = int(cnt.item())
+    assert (buf[:shift] == -7).all().item()
+    assert (buf[shift + c:shift + c + 1] == -7).all().item() or c == n  # nothing past the count
+    return out[:c].cpu().numpy()
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("n", SIZES)
+@pytest.mark.parametrize("t", [0.0, 0.001, 0.3, 1.0])
+def test_fused_select_f32_vs_oracle(mode, n, t):
+    v = gen.host(gen.F32_UNIFORM, n, seed=n % 977 + 5)
+    v[::13] = np.nan  # epsilon
+    t = float(np.float32(t))
+    pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    dv = torch.from_numpy(v).cuda()
+    got = _select(fn, dv, n, t)
+    assert len(got) == cnt_o and np.array_equal(got, pos_o)
+    with env(VD_SELECT_FUSED="0"):  # the bitmap path agrees
+        assert np.array_equal(_select(fn, dv, n, t), pos_o)
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("shift", [1, 2, 3])
+def test_fused_select_unaligned_output(mode, shift):
+    n = 5 * 8192 + 777
+    v = gen.host(gen.F32_UNIFORM, n, seed=3)
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    dv = torch.from_numpy(v).cuda()
+    for t in (0.02, 0.5, 0.99):
+        t = float(np.float32(t))
+        pos_o, _, _ = oracle.select_f32(v, t, "lt")
+        assert np.array_equal(_select(fn, dv, n, t, shift), pos_o)
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+def test_fused_select_i32_tiles_alternating_empty_and_full(mode):
+    """Tiles that select nothing next to tiles that select everything (the
+    look-back sums zero and full aggregates), against the interpreter."""
+    n = 9 * 8192 + 100
+    rng = np.random.default_rng(1)
+    a = rng.integers(-1000, 1000, n).astype(np.int32)
+    tile = np.arange(n) // 8192
+    a[tile % 3 == 0] = 5000   # never selected
+    a[tile % 3 == 1] = -5000  # always selected
+    a[::101] = -2**31         # epsilon: never selected (A9)
+    m = a == -2**31
+    p = oracle.run("p := Greater(17, v)\npos := FoldSelect(p)", v=(a.astype(np.int64), m))
+    exp = np.array([x for x in p.get("pos") if x is not None])
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    da = torch.from_numpy(a).cuda()
+    out = torch.empty(n, dtype=torch.int32, device="cuda")
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    fn([vd.column(da)], n, vd.pred([[(0, "<", 17)]]), out_pos=out, out_count=cnt)
+    k = int(cnt.item())
+    assert np.array_equal(out[:k].cpu().numpy(), exp)
