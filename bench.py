@@ -34,7 +34,7 @@ METRIC = "rows/s and achieved HBM GB/s (% of peak) for TPC-H Q1/Q6 at 1/2/4/8 B2
 
 # Algorithmic bytes per row: every
 # column each query reads, once.
-BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "selpos": 4, "c1": 4,
+BYTES_PER_ROW = {"q1": 4 + 1 + 1 + 4 * 8, "q6": 4 + 3 * 8, "select": 4, "selpos": 4, "c1": 4, "selagg": 8,
                  "q19": 4 + 3 * 8 + 1 + 1, "q9": 4 + 4 + 2 * 8, "fkjsel": 4 + 4, "q15": 24}
 L2_CAP_BYTES_PER_CLK = 6300  # B300_MICROARCH.md "LTS throughput cap" (full chip)
 
@@ -46,10 +46,12 @@ def parse():
     ap.add_argument("--warmup", type=int, default=5)
     ap.add_argument("--impl", default="voodoo", choices=["voodoo", "reference"])
     ap.add_argument("--workload", default="q1",
-                    choices=["q1", "q6", "select", "selpos", "q19", "q9", "fkjsel", "select_unfused", "fig14", "q15",
+                    choices=["q1", "q6", "select", "selagg", "selpos", "q19", "q9", "fkjsel", "fig14", "q15",
                              "c1"])
-    ap.add_argument("--chunk", type=int, default=0,
-                    help="select_unfused: rows per materialised chunk (0 = whole table; Fig 15 'Vectorized')")
+    ap.add_argument("--materialize", default="none", choices=["none", "break", "chunks"],
+                    help="selagg/q6/q1: the pipeline plan -- fused, Break (predicate materialised, Fig 8) or "
+                         "Materialize of per-chunk position lists (Fig 15 'Vectorized')")
+    ap.add_argument("--chunk", type=int, default=0, help="--materialize chunks: rows per chunk (0 = 1024)")
     ap.add_argument("--sf", type=float, default=None, help="scale factor (default: q1 100, q6 10, fkj 100)")
     ap.add_argument("--sel-mode", default="branch", choices=["branch", "predicated", "lookup"])
     ap.add_argument("--selectivity", type=float, default=0.5, help="select workload: fraction selected")
@@ -71,7 +73,7 @@ def parse():
 
 def default_sf(w):
     return {"q15": 100.0, "q1": 100.0, "q6": 10.0, "q19": 100.0, "q9": 100.0, "select": 0.0, "selpos": 0.0, "fkjsel": 0.0,
-            "select_unfused": 0.0, "fig14": 0.0}[w]
+            "selagg": 0.0, "c1": 0.0, "fig14": 0.0}[w]
 
 
 # ---------------------------------------------------------------------------
@@ -362,8 +364,6 @@ def main():
         return reference_arm(args, rank, world, sf)
     if args.workload == "selpos":
         return selpos_main(args, rank, world, local)
-    if args.workload == "select_unfused":
-        return unfused_main(args, rank, world, local)
     if args.workload == "fig14":
         return fig14_main(args, rank, world, local)
     if args.workload == "q15":
@@ -431,10 +431,16 @@ def main():
         t = torch.empty(m, dtype=torch.int64, device=dev)
         gen.device(gen.I64_UNIFORM, t.data_ptr(), m, 0, seed=args.seed + 2, p0=0, p1=10**6, stream=stream.cuda_stream)
         dims.append(t)
+    elif w == "selagg":
+        # Fig 15: sum(v2) where v1 between 0 and s, two f32 columns
+        names = ["v1", "v2"]
+        plan = plans.selagg(0.0, float(__import__("numpy").float32(args.selectivity)), sel_mode)
     else:
         names = ["v"]
         plan = plans.selsum(float(__import__("numpy").float32(args.selectivity)), sel_mode,
                             force_generic=args.generic)
+    mat = {"none": vd.VD_MAT_NONE, "break": vd.VD_MAT_BREAK, "chunks": vd.VD_MAT_CHUNKS}[args.materialize]
+    plan.materialize, plan.mat_chunk = mat, args.chunk
     for nm in names:
         if w == "fkjsel":
             c = torch.empty(n, dtype=torch.int32, device=dev)
@@ -446,8 +452,12 @@ def main():
                            stream=stream.cuda_stream)
             cols.append(c)
             continue
-        col = gen.F32_UNIFORM if nm == "v" else gen.LINEITEM_COLS[nm]
-        cols.append(make(col, n, a))
+        if nm in ("v", "v1", "v2"):
+            t = torch.empty(n, dtype=torch.float32, device=dev)
+            gen.device(gen.F32_UNIFORM, t.data_ptr(), n, a, seed=args.seed + (nm == "v2"), stream=stream.cuda_stream)
+            cols.append(t)
+            continue
+        cols.append(make(gen.LINEITEM_COLS[nm], n, a))
     torch.cuda.synchronize()
     views = [meta(t) for t in cols]
     dim_views = [meta(t) for t in dims]
@@ -531,7 +541,7 @@ def main():
     ms_per_step = elapsed_ms / steps
 
     # the step's answer: the device vd_result (merged + compacted on the GPU)
-    fl = [w == "select"] + [False] * 8
+    fl = [w in ("select", "selagg")] + [False] * 8
     result_dev = result
     result = result_dev.decode(plan, float_aggs=fl)
     if world > 1:  # cross-check against the host merge of the gathered partials
@@ -603,7 +613,7 @@ def main():
         "higher_is_better": True,
         "scaling": "strong",
         "vs_baseline": None,
-        "dtype": "f32/f64" if w == "select" else "int64",
+        "dtype": "f32/f64" if w in ("select", "selagg") else "int64",
         "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
         "config": bench_config(args, w, sf, world),
         "fragment": "generic" if args.generic else frag,
@@ -831,79 +841,6 @@ class Comm:
         if self.world > 1:
             self.dist.barrier()
             self.dist.destroy_process_group()
-
-
-def unfused_main(args, rank, world, local):
-    """Selective aggregation without fusion (Fig 15's Materialize / Break, and
-    with --chunk its 'Vectorized' cache-sized chunks): per chunk
-    select -> int32 positions (materialised), gather the values (materialised),
-    FoldSum the chunk (positions past the count are -1 = epsilon, skipped by the
-    fold), then FoldSum the chunk partials.  Compare with --workload select."""
-    import numpy as np
-    import torch
-
-    import gen
-    from paper_journals_pvldb_pirkmzm16_b200 import vd
-
-    ndev = torch.cuda.device_count()
-    torch.cuda.set_device(local % ndev)
-    dev = torch.device("cuda", local % ndev)
-    comm = Comm(world, args.dist_backend, dev)
-    stream = torch.cuda.current_stream()
-    n_total = args.rows or 10**9
-    a, b = rank * n_total // world, (rank + 1) * n_total // world
-    n = b - a
-    v = torch.empty(n, dtype=torch.float32, device=dev)
-    gen.device(gen.F32_UNIFORM, v.data_ptr(), n, a, seed=args.seed, stream=stream.cuda_stream)
-    C = args.chunk if args.chunk > 0 else n
-    nch = (n + C - 1) // C
-    t = float(np.float32(args.selectivity))
-    p = vd.pred([[(0, "<", t)]])
-    fn = vd.select_predicated if args.sel_mode == "predicated" else vd.select_branch
-    pos = torch.empty(C, dtype=torch.int32, device=dev)
-    vals = torch.empty(C, dtype=torch.float32, device=dev)
-    cnt = torch.zeros(1, dtype=torch.int64, device=dev)
-    parts = torch.zeros(nch, dtype=torch.float64, device=dev)
-    total = torch.zeros(1, dtype=torch.float64, device=dev)
-    ws = vd.alloc_ws(max(vd.workspace_bytes(vd.VD_OP_SELECT, C), vd.workspace_bytes(vd.VD_OP_FOLD, C)), dev)
-    views = [vd.column(v[k * C:min(n, (k + 1) * C)]) for k in range(nch)]
-
-    def step():
-        for k in range(nch):
-            m = views[k].len
-            pos.fill_(-1)  # materialised buffer, epsilon beyond the count
-            fn([views[k]], m, p, out_pos=pos, out_count=cnt, ws=ws, stream=stream)
-            vd.gather(views[k], pos, m, 0, vals, stream=stream)
-            pv = parts[k:k + 1]
-            vd.fold_sum(vd.column(vals, length=m), None, out=pv, ws=ws, stream=stream)
-        vd.fold_sum(vd.column(parts), None, out=total, ws=ws, stream=stream)
-
-    for _ in range(max(args.warmup, 3)):
-        step()
-    torch.cuda.synchronize()
-    steps = args.steps or 20
-    comm.barrier()
-    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    e0.record(stream)
-    for _ in range(steps):
-        step()
-    e1.record(stream)
-    torch.cuda.synchronize()
-    ms = comm.max([e0.elapsed_time(e1) / steps])[0]
-    peak, kind = hbm_peak()
-    alg = 4 * n / (ms * 1e-3) / 1e9
-    line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
-            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
-            "vs_baseline": None, "dtype": "f32/f64", "data": "synthetic (f32 U[0,1))",
-            "config": {"workload": f"select_unfused_{n_total}_s{args.selectivity:g}_chunk{C}",
-                       "sel_mode": args.sel_mode, "chunks": nch},
-            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
-                         "peak_kind": kind, "traffic": None, "kernel": "select+gather+fold (unfused)",
-                         "kernel_ms": ms},
-            "result": float(total.item()), "e2e": None}
-    if rank == 0:
-        print(json.dumps(line), flush=True)
-    comm.close()
 
 
 def fig14_main(args, rank, world, local):
@@ -1192,7 +1129,7 @@ def e2e_measure(args, torch, vd, plan, cols, views, dims, dim_views, n, dev, str
 
 def workload_rows(args, w, sf):
     import gen
-    if w in ("select", "selpos", "select_unfused"):
+    if w in ("select", "selpos", "selagg"):
         return args.rows or 10**9
     if w in ("fkjsel", "fig14"):
         return args.rows or 200_000_000
@@ -1209,11 +1146,13 @@ def bench_config(args, w, sf, world):
     name = {"q1": f"tpch_q1_sf{sf:g}", "q6": f"tpch_q6_sf{sf:g}", "q19": f"fkj_q19_sf{sf:g}",
             "q9": f"fkj_q9_sf{sf:g}", "q15": f"tpch_q15_revenue_sf{sf:g}",
             "select": f"select_f32_{n_total}_s{args.selectivity:g}",
+            "selagg": f"selagg_f32x2_{n_total}_s{args.selectivity:g}",
             "selpos": f"selpos_f32_{n_total}_s{args.selectivity:g}",
             "c1": f"c1_select_f32_{n_total}_s{args.selectivity:g}",
             "fkjsel": f"fkjsel_{n_total}x16777216_s{args.selectivity:g}"}.get(w, w)
     per_gpu = n_total // world
     return {"workload": name, "rows": n_total, "rows_per_gpu": per_gpu, "sf": sf, "sel_mode": args.sel_mode,
+            **({"materialize": args.materialize, "chunk": args.chunk} if args.materialize != "none" else {}),
             "parallelism": f"row-range x{world}" + (" + NCCL all_gather of partials" if world > 1 else ""),
             "l2": ("inputs L2-resident by design (C1): warm and cold (after a 512 MB L2 flush) reported"
                    if w == "c1" else f"inputs {per_gpu * bpr / 1e9:.1f} GB per GPU > 126 MB L2: no flush needed"),

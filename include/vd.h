@@ -171,7 +171,8 @@ typedef enum { VD_OP_SELECT = 0, VD_OP_FOLD = 1, VD_OP_SCATTER = 2, VD_OP_PIPELI
                VD_OP_PARTITION = 5, VD_OP_FOLD_SCAN = 6 } vd_op;
 /* Scratch bytes needed by `op` over n input slots (out_len for SCATTER;
  * ngroups*naggs for PIPELINE is taken from `plan`, which may be NULL
- * otherwise). */
+ * otherwise; a materialising plan also needs its intermediate vector: n
+ * bytes for VD_MAT_BREAK, 4 bytes per row + 4 per chunk for VD_MAT_CHUNKS). */
 struct vd_pipeline;
 vd_status vd_workspace_bytes(int32_t op, int64_t n, const vd_ctrl* ctrl, const struct vd_pipeline* plan,
                              size_t* bytes_host);
@@ -367,6 +368,23 @@ typedef struct {
     int64_t bias;    /* position = fk - bias (1 for 1-based keys) */
 } vd_gatherspec;
 
+/* Pipeline breakers (Table 2; Fig 8; Fig 15
+ * "Vectorized" P:L1202-1230).  The default fuses the whole chain into one
+ * kernel with no intermediate vector.  The two materialising plans split it
+ * at the operator the paper inserts:
+ *   VD_MAT_BREAK  : Break(pred) -- the predicate is evaluated fully
+ *       data-parallel and materialised in memory (one byte per row, the
+ *       workspace); a second kernel folds the rows whose flag is set.
+ *   VD_MAT_CHUNKS : Materialize(positions, Divide(Range, mat_chunk)) -- the
+ *       X100-style vectorized plan: per chunk of mat_chunk rows (one run of
+ *       the control vector) the ascending positions of the qualifying rows
+ *       are written, in order, to the chunk's slice of a position buffer in
+ *       memory (the workspace); a second loop resolves them (Gather) and
+ *       folds.  mat_chunk: a multiple of 32 in [32, 2^24] (0 = 1024).
+ * All plans return identical results (floating-point sums up to the
+ * association order). */
+typedef enum { VD_MAT_NONE = 0, VD_MAT_BREAK = 1, VD_MAT_CHUNKS = 2 } vd_materialize;
+
 typedef struct vd_pipeline {
     vd_pred pred;
     int32_t sel_mode; /* vd_sel_mode */
@@ -379,6 +397,9 @@ typedef struct vd_pipeline {
     int32_t naggs;
     int32_t force_generic; /* 1: bypass the specialised fragments (testing) */
     vd_agg aggs[VD_MAX_AGGS];
+    int32_t materialize; /* vd_materialize (0 = fused)                        */
+    int32_t reserved2;
+    int64_t mat_chunk;   /* VD_MAT_CHUNKS: rows per chunk (run of the control) */
 } vd_pipeline;
 
 /* Per-device partial result of a pipeline ("vd_partials"): a device buffer
@@ -478,7 +499,8 @@ vd_status vd_merge_partials_device(const vd_pipeline* plan, const vd_column* col
 int32_t vd_abi_struct_sizes(size_t* out, int32_t n);
 
 /* Name of the fragment the last vd_run_pipeline on this thread ran:
- * "q1_tma", "q1_ldg", "scalar_tma", "scalar_ldg", "selsum_tma", "gather_fold" or "generic". */
+ * "q1_tma", "q1_ldg", "scalar_tma", "scalar_ldg", "selsum_tma", "gather_fold",
+ * "generic", "break" or "mat_chunks" (the last two: materialising plans). */
 const char* vd_last_fragment(void);
 
 /* Number of kernel launches the last successful call on this thread

@@ -536,6 +536,18 @@ void exec_stmt(Ctx& c, const std::string& lhs, const std::string& op, const std:
         }
         out.n = n;
         c.vecs[lhs] = out;
+    } else if (op == "Materialize" || op == "Break") {
+        // Materialize(V1, V2.kp) / Break(V1, V2.kp) (Table 2):
+        // "materialize V1 in memory ... in chunks of sizes according to runs
+        // in V2.kp" / "break up V1 into segments according to the runs in
+        // V2.kp (pure tuning hint)".  Both direct HOW a program executes
+        // (where the pipeline is cut, how large the buffered chunks are), not
+        // what it computes: their value is V1.  The interpreter materialises
+        // every intermediate anyway, so it returns V1 unchanged.
+        need(2);
+        getvec(c, a[1]);  // the control vector must exist
+        if (a[0].attr.empty()) c.vecs[lhs] = getvec(c, a[0]);
+        else c.vecs[lhs] = single(a[0].attr, getcol(c, a[0], 0));
     } else if (op == "Project") {  // Project(V.kp) -- renamed to lhs
         need(1);
         c.vecs[lhs] = single(lhs, getcol(c, a[0], 0));

@@ -27,6 +27,7 @@
 #include <cmath>
 #include <cstdlib>
 #include <cstring>
+#include <type_traits>
 
 #include "vd_common.cuh"
 #include "vd_internal.h"
@@ -121,15 +122,47 @@ __device__ __forceinline__ bool gen_pred(const GenPlan& P, int64_t row) {
 constexpr int GEN_THREADS = 256;
 constexpr int GEN_WARPS = GEN_THREADS / 32;
 
+// Row source of the folding loop (vd_materialize): SRC_ROWS evaluates the
+// predicate per row (fused); SRC_FLAGS reads the predicate Break
+// materialised (one byte per row); SRC_CHUNKS walks the position lists
+// Materialize wrote per chunk of C rows (slot c*C + k, k < cnt[c]).
+enum { SRC_ROWS = 0, SRC_FLAGS = 1, SRC_CHUNKS = 2 };
+struct MatSrc {
+    const uint8_t* flags;
+    const int32_t* pos;
+    const int32_t* cnt;
+    int64_t C, nchunks;
+};
+
+// slot `it` of the folding loop -> (row, qualifies)
+template <int SRC>
+__device__ __forceinline__ bool mat_row(const GenPlan& P, const MatSrc& M, int64_t it, int64_t n_iter, int64_t n,
+                                        int64_t* row) {
+    if (SRC == SRC_ROWS) {
+        *row = it;
+        return it < n && gen_pred(P, it);
+    } else if (SRC == SRC_FLAGS) {
+        *row = it;
+        return it < n && M.flags[it] != 0;
+    } else {
+        if (it >= n_iter) { *row = 0; return false; }
+        const int64_t c = it / M.C, k = it - c * M.C;
+        const bool ok = k < (int64_t)__ldg(M.cnt + c);
+        *row = ok ? (int64_t)__ldg(M.pos + it) : 0;
+        return ok;
+    }
+}
+
 // Accumulator slot layout per (group, agg): 16 bytes (i128 or f64/i64 min-max);
 // slot [g][naggs] = row count.
-template <bool SMEM>
+template <bool SMEM, int SRC>
 __global__ void __launch_bounds__(GEN_THREADS) k_pipe_generic(const __grid_constant__ GenPlan P, int64_t n,
                                                               Slot16* __restrict__ block_parts, int nslots,
                                                               Slot16* __restrict__ gacc,
                                                               unsigned long long* __restrict__ gmask,
                                                               unsigned int* __restrict__ done, Slot16* __restrict__ out,
-                                                              unsigned long long* __restrict__ domain_err) {
+                                                              unsigned long long* __restrict__ domain_err,
+                                                              const MatSrc M, int64_t n_iter) {
     extern __shared__ Slot16 s_mem[];
     // [GEN_WARPS][32][naggs] staging, then (SMEM) [GEN_WARPS][nslots] accumulators
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
@@ -150,9 +183,9 @@ __global__ void __launch_bounds__(GEN_THREADS) k_pipe_generic(const __grid_const
     }
     __syncwarp();
     const int64_t stride = (int64_t)gridDim.x * GEN_THREADS;
-    for (int64_t base = (int64_t)blockIdx.x * GEN_THREADS + warp * 32; base < n; base += stride) {
-        const int64_t row = base + lane;
-        bool ok = row < n && gen_pred(P, row);
+    for (int64_t base = (int64_t)blockIdx.x * GEN_THREADS + warp * 32; base < n_iter; base += stride) {
+        int64_t row;
+        bool ok = mat_row<SRC>(P, M, base + lane, n_iter, n, &row);
         int64_t key = 0;
         if (ok) {
             for (int k = 0; k < P.nkey && ok; ++k) {
@@ -4211,7 +4244,7 @@ static size_t gen_smem(const vd_pipeline* p, bool smem_acc) {
 }
 static const size_t GEN_SMEM_MAX = 200 * 1024;
 
-size_t pipeline_ws_bytes(const vd_pipeline* p) {
+static size_t fold_ws_bytes_plan(const vd_pipeline* p) {
     size_t nslots = (size_t)p->ngroups * (p->naggs + 1);
     size_t grid = (size_t)grid_persistent(4);
     size_t gen = 256 + grid * nslots * sizeof(Slot16) + 2 * nslots * sizeof(Slot16) + 256;
@@ -4221,9 +4254,22 @@ size_t pipeline_ws_bytes(const vd_pipeline* p) {
     return (b + 255) & ~(size_t)255;
 }
 
-static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
-                             void* out, void* ws, cudaStream_t s, int* nl) {
-    GenPlan P;
+static int64_t mat_chunk_of(const vd_pipeline* p) { return p->mat_chunk > 0 ? p->mat_chunk : 1024; }
+
+// bytes of the materialised intermediate vector (after the fold workspace)
+static size_t mat_bytes(const vd_pipeline* p, int64_t n) {
+    if (p->materialize == VD_MAT_BREAK) return ((size_t)n + 255) & ~(size_t)255;
+    if (p->materialize == VD_MAT_CHUNKS) {
+        const int64_t C = mat_chunk_of(p), nch = (n + C - 1) / C;
+        return (((size_t)nch * C * 4 + 255) & ~(size_t)255) + (((size_t)nch * 4 + 255) & ~(size_t)255);
+    }
+    return 0;
+}
+
+size_t pipeline_ws_bytes(const vd_pipeline* p, int64_t n) { return fold_ws_bytes_plan(p) + mat_bytes(p, n); }
+
+static void build_genplan(const vd_pipeline* p, const vd_column* cols, int ncols, const vd_column* dims, GenPlan* out) {
+    GenPlan& P = *out;
     std::memset(&P, 0, sizeof(P));
     make_devpred(&p->pred, &P.pred);
     P.cols.ncols = ncols;
@@ -4262,11 +4308,16 @@ static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int nc
         }
         P.agg[a].isf = isf;
     }
+}
+
+template <int SRC>
+static vd_status launch_generic(const vd_pipeline* p, const GenPlan& P, int64_t n, int64_t n_iter, const MatSrc& M,
+                                void* out, void* ws, cudaStream_t s, int* nl) {
     const int nslots = (int)(p->ngroups * (p->naggs + 1));
     bool smem_acc = gen_smem(p, true) <= GEN_SMEM_MAX;
     size_t smem = gen_smem(p, smem_acc);
     int grid = grid_persistent(smem_acc && smem > 100 * 1024 ? 1 : 2);
-    int64_t maxg = (n + GEN_THREADS - 1) / GEN_THREADS;
+    int64_t maxg = (n_iter + GEN_THREADS - 1) / GEN_THREADS;
     if (maxg < 1) maxg = 1;
     if (grid > maxg) grid = (int)maxg;
     unsigned int* dn = (unsigned int*)ws;
@@ -4277,8 +4328,10 @@ static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int nc
     cudaError_t e = cudaMemsetAsync(ws, 0, 256, s);
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
     if (smem_acc) {
-        if (smem > 48 * 1024) cudaFuncSetAttribute(k_pipe_generic<true>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_generic<true><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn, (Slot16*)out, derr);
+        if (smem > 48 * 1024)
+            cudaFuncSetAttribute(k_pipe_generic<true, SRC>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_generic<true, SRC><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn, (Slot16*)out,
+                                                                  derr, M, n_iter);
     } else {
         // global accumulators: zero sums, +/- extremes for min/max images
         e = cudaMemsetAsync(gacc, 0, (size_t)nslots * sizeof(Slot16) + (size_t)nslots * 8, s);
@@ -4286,14 +4339,328 @@ static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int nc
         bool any_mm = false;
         for (int a = 0; a < p->naggs; ++a) any_mm |= (p->aggs[a].kind == VD_AGG_MIN || p->aggs[a].kind == VD_AGG_MAX);
         if (any_mm) { set_error("MIN/MAX with more groups than fit in shared memory"); return VD_E_UNSUPPORTED; }
-        if (smem > 48 * 1024) cudaFuncSetAttribute(k_pipe_generic<false>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        k_pipe_generic<false><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn, (Slot16*)out, derr);
+        if (smem > 48 * 1024)
+            cudaFuncSetAttribute(k_pipe_generic<false, SRC>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        k_pipe_generic<false, SRC><<<grid, GEN_THREADS, smem, s>>>(P, n, parts, nslots, gacc, gmask, dn,
+                                                                   (Slot16*)out, derr, M, n_iter);
     }
     ++*nl;
     e = cudaGetLastError();
     if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
-    set_fragment("generic");
     return VD_OK;
+}
+
+static vd_status run_generic(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n, const vd_column* dims,
+                             void* out, void* ws, cudaStream_t s, int* nl) {
+    GenPlan P;
+    build_genplan(p, cols, ncols, dims, &P);
+    MatSrc M{};
+    vd_status st = launch_generic<SRC_ROWS>(p, P, n, n, M, out, ws, s, nl);
+    if (st == VD_OK) set_fragment("generic");
+    return st;
+}
+
+// ============================================================================
+// Materialising plans (vd_materialize): Break and Materialize
+// ============================================================================
+// First loop.  A single-column interval predicate on an aligned 4-byte
+// column (the Fig 15 / C1 shape) is tested with vector loads; any other
+// predicate with the generic per-row evaluation.
+template <typename T>
+struct IvlTerm {
+    const T* p;
+    T lo, hi;
+};
+
+template <typename T, bool FAST>
+__device__ __forceinline__ bool mat_pred(const GenPlan& P, const IvlTerm<T>& t, int64_t row) {
+    if (FAST) {
+        const T v = __ldg(t.p + row);
+        return v >= t.lo && v <= t.hi;  // NaN / INT_MIN (epsilon) fail: bounds chosen on the host
+    }
+    return gen_pred(P, row);
+}
+
+// Break (Fig 8): the predicate, fully data parallel, materialised
+// as one byte per row; 4 rows per thread per step (one 32-bit store).
+template <typename T, bool FAST>
+__global__ void __launch_bounds__(256) k_mat_break(const __grid_constant__ GenPlan P, const IvlTerm<T> t, int64_t n,
+                                                   uint8_t* __restrict__ flags) {
+    const int64_t nq = (n + 3) / 4;
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    for (int64_t q = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; q < nq; q += stride) {
+        const int64_t r0 = q * 4;
+        uint32_t w = 0;
+        if (FAST && r0 + 4 <= n) {
+            const int4 x = __ldg(reinterpret_cast<const int4*>(t.p) + q);
+            T v[4];
+            memcpy(&v[0], &x.x, 4); memcpy(&v[1], &x.y, 4); memcpy(&v[2], &x.z, 4); memcpy(&v[3], &x.w, 4);
+#pragma unroll
+            for (int j = 0; j < 4; ++j) w |= (uint32_t)(v[j] >= t.lo && v[j] <= t.hi) << (8 * j);
+        } else {
+#pragma unroll
+            for (int j = 0; j < 4; ++j)
+                if (r0 + j < n) w |= (uint32_t)mat_pred<T, FAST>(P, t, r0 + j) << (8 * j);
+        }
+        if (r0 + 4 <= n) {
+            reinterpret_cast<uint32_t*>(flags)[q] = w;
+        } else {
+            for (int j = 0; r0 + j < n; ++j) flags[r0 + j] = (uint8_t)(w >> (8 * j));
+        }
+    }
+}
+
+// Materialize (Table 2; Fig 15 "Vectorized" P:L1202-1221): one
+// warp per chunk of C rows (a run of Divide(Range, C)) writes the ascending
+// positions of its qualifying rows, 32 rows per ballot, to the chunk's slice
+// pos[c*C ..] -- the position buffer is filled sequentially within the chunk
+// -- and its count to cnt[c].
+template <typename T, bool FAST>
+__global__ void __launch_bounds__(256) k_mat_chunks(const __grid_constant__ GenPlan P, const IvlTerm<T> t, int64_t n,
+                                                    int64_t C, int64_t nchunks, int32_t* __restrict__ pos,
+                                                    int32_t* __restrict__ cnt) {
+    const int lane = threadIdx.x & 31;
+    const unsigned lt = lanemask_lt();
+    const int64_t gw = ((int64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5;
+    const int64_t nw = ((int64_t)gridDim.x * blockDim.x) >> 5;
+    for (int64_t c = gw; c < nchunks; c += nw) {
+        const int64_t r0 = c * C, r1 = min(n, r0 + C);
+        int k = 0;
+        for (int64_t r = r0 + lane; r - lane < r1; r += 32) {
+            const bool f = r < r1 && mat_pred<T, FAST>(P, t, r);
+            const unsigned b = __ballot_sync(VD_FULL, f);
+            if (f) pos[r0 + k + __popc(b & lt)] = (int32_t)r;
+            k += __popc(b);
+        }
+        if (lane == 0) cnt[c] = k;
+    }
+}
+
+// Second loop of a scalar plan (one group, SUM/COUNT aggregates): the rows
+// the first loop materialised -- flags set, or the positions of each chunk
+// -- are resolved (Gather of every factor column at the position) and
+// folded per thread (int128 / f64), then warp -> CTA -> grid (the last CTA,
+// Fragment 2 of P:L929-931).
+constexpr int MF_THREADS = 256;
+
+template <int SRC>
+__global__ void __launch_bounds__(MF_THREADS) k_mat_fold(const __grid_constant__ GenPlan P, const MatSrc M, int64_t n,
+                                                         Slot16* __restrict__ parts, unsigned int* __restrict__ done,
+                                                         Slot16* __restrict__ out) {
+    const int NA = P.naggs;
+    i128 si[VD_MAX_AGGS];
+    double sf[VD_MAX_AGGS];
+#pragma unroll
+    for (int a = 0; a < VD_MAX_AGGS; ++a) { si[a] = 0; sf[a] = 0; }
+    int64_t rows = 0;
+    auto fold_row = [&](int64_t row) {
+        ++rows;
+#pragma unroll
+        for (int a = 0; a < VD_MAX_AGGS; ++a) {
+            if (a >= NA) break;
+            const GenAgg& A = P.agg[a];
+            if (A.kind == VD_AGG_COUNT) { si[a] += 1; continue; }
+            if (A.isf) {
+                double pr = 1.0;
+                bool e = false;
+                for (int f = 0; f < A.nf; ++f) {
+                    double x = 0;
+                    if (A.col[f] >= 0) {
+                        const Val c = gen_fetch(P, A.col[f], row);
+                        e |= c.eps;
+                        x = c.isf ? c.f : (double)c.i;
+                    }
+                    pr *= (double)A.a[f] + (double)A.b[f] * x;
+                }
+                if (!e) sf[a] += pr;  // an epsilon factor: the value is epsilon, skipped (A5)
+            } else {
+                i128 pr = 1;
+                bool e = false;
+                for (int f = 0; f < A.nf; ++f) {
+                    i128 x = 0;
+                    if (A.col[f] >= 0) {
+                        const Val c = gen_fetch(P, A.col[f], row);
+                        e |= c.eps;
+                        x = c.i;
+                    }
+                    pr *= (i128)A.a[f] + (i128)A.b[f] * x;
+                }
+                if (!e) si[a] += pr;
+            }
+        }
+    };
+    const int lane = threadIdx.x & 31;
+    if (SRC == SRC_FLAGS) {
+        const int64_t nq = (n + 3) / 4;
+        const int64_t stride = (int64_t)gridDim.x * MF_THREADS;
+        for (int64_t q = (int64_t)blockIdx.x * MF_THREADS + threadIdx.x; q < nq; q += stride) {
+            const int64_t r0 = q * 4;
+            uint32_t w;
+            if (r0 + 4 <= n) {
+                w = __ldg(reinterpret_cast<const uint32_t*>(M.flags) + q);
+            } else {
+                w = 0;
+                for (int j = 0; r0 + j < n; ++j) w |= (uint32_t)M.flags[r0 + j] << (8 * j);
+            }
+            for (int j = 0; j < 4; ++j)
+                if ((w >> (8 * j)) & 0xFFu) fold_row(r0 + j);
+        }
+    } else {
+        const int64_t gw = ((int64_t)blockIdx.x * MF_THREADS + threadIdx.x) >> 5;
+        const int64_t nw = ((int64_t)gridDim.x * MF_THREADS) >> 5;
+        for (int64_t c = gw; c < M.nchunks; c += nw) {  // one warp per chunk's position list
+            const int k1 = __ldg(M.cnt + c);
+            for (int k = lane; k < k1; k += 32) fold_row((int64_t)__ldg(M.pos + c * M.C + k));
+        }
+    }
+    // warp -> CTA -> grid, fixed order
+    __shared__ Slot16 s_w[MF_THREADS / 32][VD_MAX_AGGS + 1];
+    const int warp = threadIdx.x >> 5;
+    for (int a = 0; a <= NA; ++a) {
+        Slot16 v;
+        if (a < NA && P.agg[a].isf && P.agg[a].kind != VD_AGG_COUNT) {
+            put_f64(&v, warp_sum_f64(sf[a]));
+        } else {
+            put_i128(&v, warp_sum_i128(a < NA ? si[a] : (i128)rows));
+        }
+        if (lane == 0) s_w[warp][a] = v;
+    }
+    __syncthreads();
+    if (threadIdx.x <= NA) {
+        const int a = threadIdx.x;
+        const bool fl = a < NA && P.agg[a].isf && P.agg[a].kind != VD_AGG_COUNT;
+        Slot16 r = s_w[0][a];
+        for (int w = 1; w < MF_THREADS / 32; ++w) {
+            if (fl) put_f64(&r, get_f64(r) + get_f64(s_w[w][a]));
+            else put_i128(&r, get_i128(r) + get_i128(s_w[w][a]));
+        }
+        parts[(size_t)blockIdx.x * (NA + 1) + a] = r;
+    }
+    __shared__ bool s_last;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(done, 1u) == gridDim.x - 1;
+    }
+    __syncthreads();
+    if (!s_last) return;
+    __threadfence();
+    if (threadIdx.x <= NA) {
+        const int a = threadIdx.x;
+        const bool fl = a < NA && P.agg[a].isf && P.agg[a].kind != VD_AGG_COUNT;
+        Slot16 r;
+        r.lo = __ldcg(&parts[a].lo);
+        r.hi = __ldcg(&parts[a].hi);
+        for (unsigned b = 1; b < gridDim.x; ++b) {
+            Slot16 x;
+            x.lo = __ldcg(&parts[(size_t)b * (NA + 1) + a].lo);
+            x.hi = __ldcg(&parts[(size_t)b * (NA + 1) + a].hi);
+            if (fl) put_f64(&r, get_f64(r) + get_f64(x));
+            else put_i128(&r, get_i128(r) + get_i128(x));
+        }
+        out[a] = r;
+    }
+}
+
+// The predicate's fast form: <= 2 interval terms on ONE 16-byte aligned
+// f32 / i32 column (epsilon outside the bounds), else generic evaluation.
+template <typename T>
+static bool ivl_term(const vd_pipeline* p, const vd_column* cols, int ncols, IvlTerm<T>* t) {
+    if (p->ngathers != 0 || p->pred.nconj != 1 || p->pred.conj[0].nterms < 1 || p->pred.conj[0].nterms > 2)
+        return false;
+    const int c = p->pred.conj[0].terms[0].col;
+    for (int k = 0; k < p->pred.conj[0].nterms; ++k)
+        if (p->pred.conj[0].terms[k].col != c) return false;
+    if (c >= ncols || ((uintptr_t)cols[c].data & 15) != 0) return false;
+    const bool isf = std::is_same<T, float>::value;
+    if (cols[c].dtype != (isf ? VD_F32 : VD_I32)) return false;
+    t->p = (const T*)cols[c].data;
+    if (isf) {
+        int32_t fcmp[2] = {-1, -1};
+        double fc[2] = {0, 0};
+        for (int k = 0; k < p->pred.conj[0].nterms; ++k) {
+            fcmp[k] = p->pred.conj[0].terms[k].cmp;
+            fc[k] = p->pred.conj[0].terms[k].fval;
+        }
+        float lo, hi;
+        if (!f32_interval(fcmp, fc, &lo, &hi)) return false;
+        memcpy(&t->lo, &lo, 4);
+        memcpy(&t->hi, &hi, 4);
+        return true;
+    }
+    int64_t lo = (int64_t)INT32_MIN + 1, hi = INT32_MAX;  // epsilon never qualifies (A9)
+    for (int k = 0; k < p->pred.conj[0].nterms; ++k)
+        if (!term_interval(p->pred.conj[0].terms[k], &lo, &hi)) return false;
+    if (lo > hi) { lo = 1; hi = 0; }
+    int32_t l32 = (int32_t)lo, h32 = (int32_t)hi;
+    memcpy(&t->lo, &l32, 4);
+    memcpy(&t->hi, &h32, 4);
+    return true;
+}
+
+template <typename T, bool FAST>
+static void launch_mat_first(const vd_pipeline* p, const GenPlan& P, const IvlTerm<T>& t, int64_t n, const MatSrc& M,
+                             cudaStream_t s, int* nl) {
+    const int64_t grid = grid_persistent(8);
+    if (p->materialize == VD_MAT_BREAK)
+        k_mat_break<T, FAST><<<(int)std::max<int64_t>(1, std::min<int64_t>(grid, (n + 1023) / 1024)), 256, 0, s>>>(
+            P, t, n, const_cast<uint8_t*>(M.flags));
+    else
+        k_mat_chunks<T, FAST><<<(int)std::max<int64_t>(1, std::min<int64_t>(grid, (M.nchunks + 7) / 8)), 256, 0, s>>>(
+            P, t, n, M.C, M.nchunks, const_cast<int32_t*>(M.pos), const_cast<int32_t*>(M.cnt));
+    ++*nl;
+}
+
+static vd_status run_materialized(const vd_pipeline* p, const vd_column* cols, int ncols, int64_t n,
+                                  const vd_column* dims, void* out, void* ws, cudaStream_t s, int* nl) {
+    GenPlan P;
+    build_genplan(p, cols, ncols, dims, &P);
+    char* mat = (char*)ws + fold_ws_bytes_plan(p);
+    MatSrc M{};
+    int64_t n_iter = n;
+    if (p->materialize == VD_MAT_BREAK) {
+        M.flags = (const uint8_t*)mat;
+    } else {
+        M.C = mat_chunk_of(p);
+        M.nchunks = (n + M.C - 1) / M.C;
+        M.pos = (const int32_t*)mat;
+        M.cnt = (const int32_t*)(mat + (((size_t)M.nchunks * M.C * 4 + 255) & ~(size_t)255));
+        n_iter = M.nchunks * M.C;
+    }
+    // first loop: the pipeline breaker writes its vector to memory
+    IvlTerm<float> tf{};
+    IvlTerm<int32_t> ti{};
+    if (ivl_term<float>(p, cols, ncols, &tf)) launch_mat_first<float, true>(p, P, tf, n, M, s, nl);
+    else if (ivl_term<int32_t>(p, cols, ncols, &ti)) launch_mat_first<int32_t, true>(p, P, ti, n, M, s, nl);
+    else launch_mat_first<float, false>(p, P, tf, n, M, s, nl);
+    cudaError_t e = cudaGetLastError();
+    if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    // second loop: fold the materialised rows
+    const int src = p->materialize == VD_MAT_BREAK ? SRC_FLAGS : SRC_CHUNKS;
+    bool simple = p->nkeyparts == 0 && p->ngroups == 1;
+    for (int a = 0; a < p->naggs; ++a)
+        simple = simple && (p->aggs[a].kind == VD_AGG_SUM || p->aggs[a].kind == VD_AGG_COUNT);
+    vd_status st = VD_OK;
+    if (simple) {
+        unsigned int* dn = (unsigned int*)ws;
+        Slot16* parts = (Slot16*)((char*)ws + 256);
+        e = cudaMemsetAsync(dn, 0, 4, s);
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+        const int64_t work = src == SRC_FLAGS ? (n + 3) / 4 : M.nchunks * 32;
+        const int grid = (int)std::max<int64_t>(
+            1, std::min<int64_t>(grid_persistent(4), (work + MF_THREADS - 1) / MF_THREADS));
+        if (src == SRC_FLAGS) k_mat_fold<SRC_FLAGS><<<grid, MF_THREADS, 0, s>>>(P, M, n, parts, dn, (Slot16*)out);
+        else k_mat_fold<SRC_CHUNKS><<<grid, MF_THREADS, 0, s>>>(P, M, n, parts, dn, (Slot16*)out);
+        ++*nl;
+        e = cudaGetLastError();
+        if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
+    } else if (src == SRC_FLAGS) {
+        st = launch_generic<SRC_FLAGS>(p, P, n, n_iter, M, out, ws, s, nl);
+    } else {
+        st = launch_generic<SRC_CHUNKS>(p, P, n, n_iter, M, out, ws, s, nl);
+    }
+    if (st == VD_OK) set_fragment(p->materialize == VD_MAT_BREAK ? "break" : "mat_chunks");
+    return st;
 }
 
 vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncols, int64_t n, const vd_column* dims,
@@ -4305,6 +4672,7 @@ vd_status run_pipeline(const vd_pipeline* p, const vd_column* cols, int32_t ncol
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
         return VD_OK;
     }
+    if (p->materialize != VD_MAT_NONE) return run_materialized(p, cols, ncols, n, dims, out, ws, s, nl);
     if (!p->force_generic) {
         bool done = false;
         vd_status st = try_q1(p, cols, ncols, n, out, ws, s, nl, &done);

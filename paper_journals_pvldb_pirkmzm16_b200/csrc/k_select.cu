@@ -500,35 +500,106 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
 }
 
 // ---- fused single-pass selection (TMA ring + decoupled look-back) -------------
-// One pass, no materialised predicate: a producer warp claims tiles of
-// SF_CW x 1024 rows IN ORDER from a global counter (every predecessor of a
-// claimed tile is claimed by a running CTA: forward progress for the
-// look-back) and streams them into an SF_STAGES-deep mbarrier ring with 1D
-// bulk copies; consumer warp w turns 1024 rows of the tile into 32 ballots
-// held in registers (bit L of ballot 4q+j <-> row q*128 + 32j + L: each
-// ballot is directly a row-ordered 32-bit word) and releases the ring slot
-// at once, so HBM keeps streaming while the warp waits for its offset.
-// Warp 0 turns the warp counts into the tile aggregate and runs the
-// decoupled look-back (Merrill & Garland's single-pass scan) over per-tile
-// status words; then every warp stages its positions in shared memory --
-// branching: qualifying lanes store at their rank; predicated: cursor
-// arithmetic, every row stored at the cursor, the cursor advancing by the
-// predicate -- and streams the ascending run out with 16-byte
-// stores.  Two CTAs per SM, so one CTA's look-back wait overlaps the
-// other's work.  Replaces the 3-launch bitmap path (flag pass, scan,
-// position pass) for single interval terms on 4-byte columns.
-constexpr int SF_CW = 8;
-constexpr int SF_THREADS = SF_CW * 32 + 32;
+// One pass, no materialised predicate.  Warp roles of a CTA (one per SM):
+//   producer  : claims tiles of SF_CW x 1024 rows IN ORDER from a global
+//               counter (every predecessor of a claimed tile is claimed by a
+//               running CTA: forward progress) and streams them into an
+//               SF_STAGES-deep mbarrier ring with 1D bulk copies;
+//   consumers : warp w turns its 1024 rows of tile i into 32 ballots (bit L
+//               of ballot 4q+j <-> row q*128 + 32j + L: each ballot is a
+//               row-ordered 32-bit word), releases the ring slot, publishes
+//               its count -- and only then writes the positions of tile i-1,
+//               whose offset the look-back warp has resolved meanwhile;
+//   look-back : sums tile i's warp counts, publishes the tile aggregate at
+//               once and runs the decoupled look-back (single-pass scan over
+//               per-tile status words) for the tile's global offset.
+// Counting never waits for a look-back, so every claimed tile publishes its
+// aggregate as soon as its data lands and the inclusive-prefix frontier
+// trails the newest tile by about one L2 round trip of tiles -- within one
+// 128-tile look-back window (a coupled design, where a warp counts tile i+1
+// only after tile i's offset is known, let unpublished claimed tiles stall
+// every successor's look-back: 7.6-8.1 ms for 1e9 rows).
+// Positions: branching -- qualifying lanes store at their rank; predicated --
+// cursor arithmetic, every row stored at the cursor and the cursor advanced
+// by the predicate; then the ascending run streams out with
+// 16-byte stores.  Replaces the 3-launch bitmap path for single interval
+// terms on 4-byte columns.
+constexpr int SF_CW = 16;
+constexpr int SF_THREADS = SF_CW * 32 + 64;   // + producer warp + look-back warp
 constexpr int SF_STAGES = 2;
 constexpr int SF_ROWS = SF_CW * 1024;         // rows per tile
 constexpr int SF_STG = 1024 + 128 + 8;        // per-warp position stage (ints)
 
-__device__ __forceinline__ void bar_consumers() {
-    asm volatile("bar.sync 1, %0;" ::"n"(SF_CW * 32) : "memory");
+struct SfShared {
+    uint64_t full[SF_STAGES], empty[SF_STAGES];
+    uint64_t cnt_bar[2], base_bar[2];
+    int64_t s_tile[SF_STAGES];
+    int64_t lb_tile[2];
+    int64_t base[2];
+    int cnt[2][SF_CW];
+    int woff[2][SF_CW];
+    uint32_t bal[2][SF_CW][32];
+};
+
+template <int MODE>
+__device__ __forceinline__ void sf_write_positions(const uint32_t* __restrict__ bal, int64_t row_w, int64_t g0,
+                                                   int32_t* __restrict__ out, int32_t* __restrict__ sw, int lane,
+                                                   unsigned lt) {
+    uint32_t bw[32];
+#pragma unroll
+    for (int k = 0; k < 32; k += 4) {
+        const uint4 x = *reinterpret_cast<const uint4*>(bal + k);  // broadcast
+        bw[k] = x.x; bw[k + 1] = x.y; bw[k + 2] = x.z; bw[k + 3] = x.w;
+    }
+    // stage index a + k <-> output g0 + k, a = the output's misalignment in
+    // words, so stage groups of 4 are 16-byte output groups
+    const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+    int cur = a;
+#pragma unroll
+    for (int q = 0; q < 8; ++q) {
+        const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
+        int pre = cur;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            const uint32_t w = bw[4 * q + j];
+            const int f = (w >> lane) & 1u;
+            const int r = __popc(w & lt);
+            const int32_t row = (int32_t)(row_w + q * 128 + j * 32 + lane);
+            if (MODE == 0) {
+                if (f) sw[pre + r] = row;
+            } else {
+                // cursor arithmetic: unconditional store; rows that do not
+                // qualify land past the block's count and are overwritten
+                const int sel_before = pre - cur + r;
+                const int k = f ? pre + r : cur + cq + (j * 32 + lane - sel_before);
+                sw[k] = row;
+            }
+            pre += __popc(w);
+        }
+        cur += cq;
+    }
+    __syncwarp();
+    const int total = cur - a;
+    const int ngr = (a + total + 3) >> 2;
+    int32_t* ob = out + g0 - a;  // 16-byte aligned
+    for (int v = lane; v < ngr; v += 32) {
+        const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
+        if (4 * v >= a && 4 * v + 4 <= a + total) {
+            __stcs(reinterpret_cast<int4*>(ob) + v, x);
+        } else {
+            const int32_t xs[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+            for (int e = 0; e < 4; ++e) {
+                const int k = 4 * v + e;
+                if (k >= a && k < a + total) __stcs(ob + k, xs[e]);
+            }
+        }
+    }
+    __syncwarp();
 }
 
 template <int MODE, typename T>
-__global__ void __launch_bounds__(SF_THREADS, 2) k_sel_fused(const T* __restrict__ col, T lo, T hi, int64_t n,
+__global__ void __launch_bounds__(SF_THREADS, 1) k_sel_fused(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                              int64_t ntiles, int32_t* __restrict__ out,
                                                              int64_t* __restrict__ out_count,
                                                              uint64_t* __restrict__ status,
@@ -536,17 +607,17 @@ __global__ void __launch_bounds__(SF_THREADS, 2) k_sel_fused(const T* __restrict
     constexpr uint32_t TB = SF_ROWS * sizeof(T);
     extern __shared__ __align__(128) uint8_t smem[];
     int32_t* stage = reinterpret_cast<int32_t*>(smem + (size_t)SF_STAGES * TB);
-    uint64_t* full = reinterpret_cast<uint64_t*>(stage + SF_CW * SF_STG);
-    uint64_t* empty = full + SF_STAGES;
-    int64_t* s_tile = reinterpret_cast<int64_t*>(empty + SF_STAGES);
-    __shared__ int s_cnt[SF_CW], s_woff[SF_CW];
-    __shared__ int64_t s_base;
+    SfShared& S = *reinterpret_cast<SfShared*>(stage + SF_CW * SF_STG);
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int64_t nfull = n / SF_ROWS;  // tiles loaded by TMA; the ragged last one by LDG
     if (threadIdx.x == 0) {
         for (int i = 0; i < SF_STAGES; ++i) {
-            mbar_init(&full[i], 1);
-            mbar_init(&empty[i], SF_CW);
+            mbar_init(&S.full[i], 1);
+            mbar_init(&S.empty[i], SF_CW);
+        }
+        for (int i = 0; i < 2; ++i) {
+            mbar_init(&S.cnt_bar[i], SF_CW);
+            mbar_init(&S.base_bar[i], 1);
         }
         fence_mbar_init();
     }
@@ -558,133 +629,115 @@ __global__ void __launch_bounds__(SF_THREADS, 2) k_sel_fused(const T* __restrict
             int st = 0;
             uint32_t ph = 0;
             for (int64_t it = 0;; ++it) {
-                if (it >= SF_STAGES) mbar_wait(&empty[st], ph ^ 1u);
+                if (it >= SF_STAGES) mbar_wait(&S.empty[st], ph ^ 1u);
                 const int64_t tile = (int64_t)atomicAdd(tile_ctr, 1ull);
                 if (tile >= ntiles) {
-                    s_tile[st] = -1;
-                    mbar_arrive(&full[st]);
+                    S.s_tile[st] = -1;
+                    mbar_arrive(&S.full[st]);
                     break;
                 }
-                s_tile[st] = tile;
+                S.s_tile[st] = tile;
                 if (tile < nfull) {
-                    mbar_expect_tx(&full[st], TB);
-                    tma_load_1d(smem + (size_t)st * TB, col + tile * SF_ROWS, TB, &full[st], pol);
+                    mbar_expect_tx(&S.full[st], TB);
+                    tma_load_1d(smem + (size_t)st * TB, col + tile * SF_ROWS, TB, &S.full[st], pol);
                 } else {
-                    mbar_arrive(&full[st]);  // partial tile: the consumers read it from global memory
+                    mbar_arrive(&S.full[st]);  // partial tile: the consumers read it from global memory
                 }
                 if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
             }
         }
         return;
     }
-    const unsigned lt = lanemask_lt();
-    int32_t* sw = stage + warp * SF_STG;
-    int st = 0;
-    uint32_t ph = 0;
-    for (;;) {
-        mbar_wait(&full[st], ph);
-        const int64_t tile = s_tile[st];
-        if (tile < 0) break;
-        const int64_t row_w = tile * SF_ROWS + (int64_t)warp * 1024;
-        // ---- flags -> 32 row-ordered ballot words ----
-        uint32_t bw[32];
-        if (tile < nfull) {
-            const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
-#pragma unroll
-            for (int k = 0; k < 32; ++k) {
-                const T v = src[k * 32 + lane];
-                bw[k] = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN (epsilon) fails
-            }
-        } else {
-#pragma unroll
-            for (int k = 0; k < 32; ++k) {
-                const int64_t r = row_w + k * 32 + lane;
-                bool f = false;
-                if (r < n) {
-                    const T v = __ldg(col + r);
-                    f = v >= lo && v <= hi;
-                }
-                bw[k] = __ballot_sync(VD_FULL, f);
-            }
-        }
-        __syncwarp();
-        if (lane == 0) mbar_arrive(&empty[st]);  // slot free: only the ballots are needed from here
-        if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
-        int cnt = 0;
-#pragma unroll
-        for (int k = 0; k < 32; ++k) cnt += __popc(bw[k]);
-        // ---- tile offset: warp counts -> aggregate -> decoupled look-back ----
-        if (lane == 0) s_cnt[warp] = cnt;
-        bar_consumers();
-        if (warp == 0) {
-            const int v = lane < SF_CW ? s_cnt[lane] : 0;
+    if (warp == SF_CW + 1) {
+        // ---- look-back: tile aggregate -> published -> global offset ----
+        for (int64_t i = 0;; ++i) {
+            const int sl = (int)(i & 1);
+            mbar_wait(&S.cnt_bar[sl], (uint32_t)((i >> 1) & 1));
+            const int64_t tile = S.lb_tile[sl];
+            if (tile < 0) break;
+            const int v = lane < SF_CW ? S.cnt[sl][lane] : 0;
             int incl = v;
 #pragma unroll
             for (int o = 1; o < SF_CW; o <<= 1) {
                 const int u = __shfl_up_sync(VD_FULL, incl, o);
                 if (lane >= o) incl += u;
             }
-            if (lane < SF_CW) s_woff[lane] = incl - v;
+            if (lane < SF_CW) S.woff[sl][lane] = incl - v;
             const int64_t agg = __shfl_sync(VD_FULL, incl, SF_CW - 1);
             const int64_t base = lookback_exclusive_w128(status, tile, agg, lane);
             if (lane == 0) {
-                s_base = base;
+                S.base[sl] = base;
                 if (tile == ntiles - 1) *out_count = base + agg;
+                mbar_arrive(&S.base_bar[sl]);
             }
+            __syncwarp();
         }
-        bar_consumers();
-        const int64_t g0 = s_base + s_woff[warp];
-        // ---- positions -> stage (ascending), then 16-byte streaming stores ----
-        // stage index a + k <-> output g0 + k, a = the output's misalignment
-        // in words, so stage groups of 4 are 16-byte output groups
-        const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
-        int cur = a;
+        return;
+    }
+    // ---- consumers ----
+    const unsigned lt = lanemask_lt();
+    int32_t* sw = stage + warp * SF_STG;
+    int st = 0;
+    uint32_t ph = 0;
+    int64_t prev_tile = -1;
+    for (int64_t i = 0;; ++i) {
+        const int sl = (int)(i & 1);
+        mbar_wait(&S.full[st], ph);
+        const int64_t tile = S.s_tile[st];
+        if (tile >= 0) {
+            const int64_t row_w = tile * SF_ROWS + (int64_t)warp * 1024;
+            uint32_t* mybal = S.bal[sl][warp];
+            int cnt = 0;
+            if (tile < nfull) {
+                const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
 #pragma unroll
-        for (int q = 0; q < 8; ++q) {
-            const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
-            int pre = cur;
-#pragma unroll
-            for (int j = 0; j < 4; ++j) {
-                const uint32_t w = bw[4 * q + j];
-                const int f = (w >> lane) & 1u;
-                const int r = __popc(w & lt);
-                const int32_t row = (int32_t)(row_w + q * 128 + j * 32 + lane);
-                if (MODE == 0) {
-                    if (f) sw[pre + r] = row;
-                } else {
-                    // cursor arithmetic: unconditional store; rows that do not
-                    // qualify land past the block's count and are overwritten
-                    const int sel_before = pre - cur + r;
-                    const int k = f ? pre + r : cur + cq + (j * 32 + lane - sel_before);
-                    sw[k] = row;
+                for (int k = 0; k < 32; ++k) {
+                    const T v = src[k * 32 + lane];
+                    const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN (epsilon) fails
+                    if (lane == k) mybal[k] = b;
+                    cnt += __popc(b);
                 }
-                pre += __popc(w);
-            }
-            cur += cq;
-        }
-        __syncwarp();
-        const int total = cur - a;
-        const int ngr = (a + total + 3) >> 2;
-        int32_t* ob = out + g0 - a;  // 16-byte aligned
-        for (int v = lane; v < ngr; v += 32) {
-            const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
-            if (4 * v >= a && 4 * v + 4 <= a + total) {
-                __stcs(reinterpret_cast<int4*>(ob) + v, x);
             } else {
-                const int32_t xs[4] = {x.x, x.y, x.z, x.w};
 #pragma unroll
-                for (int e = 0; e < 4; ++e) {
-                    const int k = 4 * v + e;
-                    if (k >= a && k < a + total) __stcs(ob + k, xs[e]);
+                for (int k = 0; k < 32; ++k) {
+                    const int64_t r = row_w + k * 32 + lane;
+                    bool f = false;
+                    if (r < n) {
+                        const T v = __ldg(col + r);
+                        f = v >= lo && v <= hi;
+                    }
+                    const uint32_t b = __ballot_sync(VD_FULL, f);
+                    if (lane == k) mybal[k] = b;
+                    cnt += __popc(b);
                 }
             }
+            __syncwarp();
+            if (lane == 0) {
+                mbar_arrive(&S.empty[st]);  // slot free: only the ballots are needed from here
+                S.cnt[sl][warp] = cnt;
+                if (warp == 0) S.lb_tile[sl] = tile;
+            }
+        } else if (warp == 0 && lane == 0) {
+            S.lb_tile[sl] = -1;  // tells the look-back warp to stop
         }
         __syncwarp();
+        if (lane == 0) mbar_arrive(&S.cnt_bar[sl]);
+        if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
+        // positions of the previous tile, whose offset is resolved by now
+        if (prev_tile >= 0) {
+            const int ps = sl ^ 1;
+            mbar_wait(&S.base_bar[ps], (uint32_t)(((i - 1) >> 1) & 1));
+            const int64_t g0 = S.base[ps] + S.woff[ps][warp];
+            sf_write_positions<MODE>(S.bal[ps][warp], prev_tile * SF_ROWS + (int64_t)warp * 1024, g0, out, sw, lane,
+                                     lt);
+        }
+        if (tile < 0) break;
+        prev_tile = tile;
     }
 }
 
 static size_t sel_fused_smem(size_t tsize) {
-    return (size_t)SF_STAGES * SF_ROWS * tsize + (size_t)SF_CW * SF_STG * 4 + 2 * SF_STAGES * 8 + SF_STAGES * 8;
+    return (size_t)SF_STAGES * SF_ROWS * tsize + (size_t)SF_CW * SF_STG * 4 + sizeof(SfShared);
 }
 
 // VD_SELECT_FUSED=0 keeps the bitmap path (comparison runs)

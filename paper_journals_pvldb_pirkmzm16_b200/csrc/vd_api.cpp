@@ -324,7 +324,8 @@ vd_status vd_workspace_bytes(int32_t op, int64_t n, const vd_ctrl* ctrl, const s
         if (!plan) return VD_E_NULL;
         if (plan->ngroups < 1 || plan->ngroups > VD_MAX_GROUPS || plan->naggs < 0 || plan->naggs > VD_MAX_AGGS)
             return VD_E_ARG;
-        *bytes = pipeline_ws_bytes(plan);
+        if (plan->materialize < VD_MAT_NONE || plan->materialize > VD_MAT_CHUNKS) return VD_E_ARG;
+        *bytes = pipeline_ws_bytes(plan, n);
         return VD_OK;
     default: set_error("unknown op"); return VD_E_ARG;
     }
@@ -649,7 +650,16 @@ vd_status vd_run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_
         for (int f = 0; f < g.nfactors; ++f)
             if (g.f[f].col < -1 || g.f[f].col >= nref) { set_error("factor column out of range"); return VD_E_ARG; }
     }
-    if ((st = check_ws(ws, ws_bytes, pipeline_ws_bytes(plan))) != VD_OK) return st;
+    if (plan->materialize < VD_MAT_NONE || plan->materialize > VD_MAT_CHUNKS) {
+        set_error("materialize: VD_MAT_NONE / VD_MAT_BREAK / VD_MAT_CHUNKS");
+        return VD_E_ARG;
+    }
+    if (plan->materialize == VD_MAT_CHUNKS && plan->mat_chunk != 0 &&
+        (plan->mat_chunk < 32 || plan->mat_chunk > (1 << 24) || plan->mat_chunk % 32 != 0)) {
+        set_error("mat_chunk: a multiple of 32 in [32, 2^24] (0 = 1024)");
+        return VD_E_ARG;
+    }
+    if ((st = check_ws(ws, ws_bytes, pipeline_ws_bytes(plan, n))) != VD_OK) return st;
     if ((st = check_device()) != VD_OK) return st;
     int nl = 0;
     st = run_pipeline(plan, cols, ncols, n, dims, ndims, out, ws, ws_bytes, (cudaStream_t)stream, &nl);

@@ -95,7 +95,7 @@ cudaError_t launch_partition(const vd_column& v, int64_t from, int64_t npiv, int
                              int64_t* out_counts, void* ws, cudaStream_t s, int* nlaunch);
 
 // k_pipeline.cu
-size_t pipeline_ws_bytes(const vd_pipeline* plan);
+size_t pipeline_ws_bytes(const vd_pipeline* plan, int64_t n);
 vd_status run_pipeline(const vd_pipeline* plan, const vd_column* cols, int32_t ncols, int64_t n,
                        const vd_column* dims, int32_t ndims, void* out, void* ws, size_t ws_bytes, cudaStream_t s,
                        int* nlaunch);

@@ -52,6 +52,16 @@ def selsum(t: float, sel_mode=VD_SEL_BRANCH, force_generic=False):
                     force_generic=force_generic)
 
 
+def selagg(lo: float, hi: float, sel_mode=VD_SEL_BRANCH, materialize=0, mat_chunk=0):
+    """Fig 15's selective aggregation:
+    SELECT sum(v2) FROM t WHERE v1 BETWEEN lo AND hi, over columns [v1, v2]
+    (f32, f64 accumulation) + count.  materialize / mat_chunk pick the plan:
+    fused (branching / predicated), Break, or the Vectorized plan's
+    Materialize of per-chunk position lists."""
+    return pipeline(pred_=pred([[(0, ">=", float(lo)), (0, "<=", float(hi))]]), sel_mode=sel_mode,
+                    aggs=[("sum", [1]), ("count",)], materialize=materialize, mat_chunk=mat_chunk)
+
+
 # the three branches of TPC-H Q19: brand, containers, quantity lower bound
 # (the upper is +10), maximum p_size
 Q19_BRANCHES = [("Brand#12", ["SM CASE", "SM BOX", "SM PACK", "SM PKG"], 1, 5),

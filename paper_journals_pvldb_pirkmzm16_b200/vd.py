@@ -34,6 +34,7 @@ VD_SEL_BRANCH, VD_SEL_PREDICATED, VD_SEL_PREDICATED_LOOKUP = 0, 1, 2
 VD_OP_SELECT, VD_OP_FOLD, VD_OP_SCATTER, VD_OP_PIPELINE, VD_OP_FOLD_SELECT, VD_OP_PARTITION, VD_OP_FOLD_SCAN = range(7)
 VD_AGG_SUM, VD_AGG_COUNT, VD_AGG_MIN, VD_AGG_MAX = range(4)
 VD_SCATTER_UNIQUE = 1
+VD_MAT_NONE, VD_MAT_BREAK, VD_MAT_CHUNKS = 0, 1, 2
 VD_COL_NOEPS = 1
 VD_MAX_TERMS, VD_MAX_CONJ, VD_MAX_AGGS, VD_MAX_FACTORS, VD_MAX_GATHERS, VD_MAX_KEYPARTS = 8, 4, 8, 3, 4, 3
 VD_WS_DOMAIN_ERRORS_OFFSET = 128
@@ -88,7 +89,8 @@ class vd_pipeline(Structure):
     _fields_ = [("pred", vd_pred), ("sel_mode", c_int32), ("ngathers", c_int32),
                 ("gathers", vd_gatherspec * VD_MAX_GATHERS), ("nkeyparts", c_int32), ("reserved", c_int32),
                 ("key", vd_keypart * VD_MAX_KEYPARTS), ("ngroups", c_int64), ("naggs", c_int32),
-                ("force_generic", c_int32), ("aggs", vd_agg * VD_MAX_AGGS)]
+                ("force_generic", c_int32), ("aggs", vd_agg * VD_MAX_AGGS), ("materialize", c_int32),
+                ("reserved2", c_int32), ("mat_chunk", c_int64)]
 
 
 class vd_result(Structure):
@@ -477,8 +479,12 @@ def partition(v: vd_column, pivot_from, npivots, out_pos, out_bucket_counts=None
 
 # ---- a7-a9 fused pipeline ----------------------------------------------------------------------
 def pipeline(*, pred_: Optional[vd_pred] = None, sel_mode: int = VD_SEL_BRANCH, gathers=(), key=(), ngroups=1,
-             aggs=(), force_generic=False) -> vd_pipeline:
+             aggs=(), force_generic=False, materialize: int = VD_MAT_NONE, mat_chunk: int = 0) -> vd_pipeline:
     """Build a vd_pipeline.
+
+    materialize: VD_MAT_NONE (fused), VD_MAT_BREAK (the predicate
+    materialised, Fig 8's break) or VD_MAT_CHUNKS (per-chunk position lists
+    of mat_chunk rows, Fig 15's vectorized plan).
 
     gathers: [(fk_col, dim_col, bias)]; key: [(col, fn, sub, mult)] (fn 0 identity, 1 year);
     aggs: [("sum", [(col, a, b), ...]) | ("count",) | ("min", [...]) | ("max", [...])], factor = a + b*col
@@ -506,6 +512,8 @@ def pipeline(*, pred_: Optional[vd_pred] = None, sel_mode: int = VD_SEL_BRANCH, 
                 f = (f, 0, 1)
             p.aggs[i].f[j].col, p.aggs[i].f[j].a, p.aggs[i].f[j].b = f
     p.force_generic = int(force_generic)
+    p.materialize = int(materialize)
+    p.mat_chunk = int(mat_chunk)
     return p
 
 

@@ -61,8 +61,29 @@ def fig14():
                 print(json.dumps(d), flush=True)
 
 
+def fig15m():
+    """Fig 15 on B200 through the library's plans: selective
+    aggregation sum(v2) where v1 between 0 and s over two 1e9-row f32
+    columns -- fused branching / predicated, Break (predicate materialised),
+    and the Vectorized plan (Materialize of per-chunk position lists)."""
+    for s in SEL:
+        for mat, chunk in (("none", 0), ("break", 0), ("chunks", 1024), ("chunks", 65536)):
+            for mode in ("branch", "predicated"):
+                cmd = [sys.executable, os.path.join(ROOT, "bench.py"), "--workload", "selagg", "--selectivity", str(s),
+                       "--sel-mode", mode, "--materialize", mat, "--chunk", str(chunk), "--steps", "20",
+                       "--no-cpu-baseline", "--no-e2e"]
+                out = subprocess.run(cmd, capture_output=True, text=True, timeout=600)
+                line = out.stdout.strip().splitlines()[-1] if out.stdout.strip() else "{}"
+                d = json.loads(line)
+                d["_sel"] = s
+                d["_mode"] = f"{mode}/{mat}" + (f"/{chunk}" if mat == "chunks" else "")
+                print(json.dumps(d), flush=True)
+
+
 def main():
     what = sys.argv[1]
+    if what == "fig15m":
+        return fig15m()
     if what == "table":
         return table(sys.argv[2:])
     if what == "fig14":

@@ -73,7 +73,8 @@ def test_device_merge_equals_host_merge_synthetic(ngroups, nparts):
         for g in range(ngroups):
             rows = int(rng.integers(1, 1000)) if rng.random() < 0.6 else 0
             if rows:
-                vals += [int(rng.integers(-2**100, 2**100)), float(rng.random() * 1e6),
+                big = int(rng.integers(-2**62, 2**62)) * 2**38 + int(rng.integers(0, 2**38))  # ~2^100
+                vals += [big, float(rng.random() * 1e6),
                          int(rng.integers(-2**62, 2**62)), int(rng.integers(-2**62, 2**62)), rows, rows]
             else:
                 vals += [0, 0.0, 0, 0, 0, 0]

@@ -126,3 +126,35 @@ def test_fig1_branching_equals_predicated_positions():
         # brute-force layer agrees
         pos, c, _ = oracle.select_f32(v, float(np.float32(t)), "lt")
         assert c == cur and pos.tolist() == got
+
+
+@pytest.mark.parametrize("chunk", [1, 32, 1000, 4096, 10**6])
+def test_fig15_materialize_and_break_leave_values_unchanged(chunk):
+    """Materialize / Break (Table 2) direct how a program runs,
+    not what it computes: the Vectorized plan (per-chunk position lists
+    materialised, chunks = runs of Divide(Range, C)) and the Break plan equal
+    the fused plan and a brute-force loop over the same f32 columns (sum of
+    v2 where lo <= v1 <= hi, long double vs exact rational tolerance)."""
+    import numpy as np
+
+    import gen
+    from oracle import programs
+    n = 20011
+    v1 = gen.host(gen.F32_UNIFORM, n, seed=7)
+    v2 = gen.host(gen.F32_UNIFORM, n, seed=8)
+    lo, hi = np.float32(0.25), np.float32(0.6)
+    m = (v1 >= lo) & (v1 <= hi)
+    from fractions import Fraction
+    exact = sum(Fraction(float(x)) for x in v2[m])
+    # v1 >= lo <=> Greater(v1, pred(lo)); v1 <= hi <=> Greater(succ(hi), v1) on f32 values
+    lom = float(np.nextafter(lo, np.float32(-1)))
+    hip = float(np.nextafter(hi, np.float32(2)))
+    res = []
+    for prog in (programs.FIG15_FUSED, programs.FIG15_VECTORIZED, programs.FIG15_BREAK):
+        p = oracle.run(prog.format(lom=lom.hex(), hip=hip.hex(), chunk=chunk), input__v1=v1, input__v2=v2)
+        t, r, _ = p.get_float_exact("total")
+        res.append((t[0] + r[0], p.get("count")[0]))
+    for tot, cnt in res:
+        assert cnt == int(m.sum())
+        assert abs(Fraction(tot) - exact) <= Fraction(1, 10**9) * exact
+    assert res[0] == res[2]  # Break: the same single fold order
