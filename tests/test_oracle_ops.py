@@ -210,3 +210,35 @@ def test_foldscan_inclusive_restart_reading_A27():
     v = np.array([1, 2, 3, 4, 5, 6])
     p = oracle.run("s := FoldScan(c, v)", c=c, v=v)
     assert p.get("s") == [1, 3, 6, 4, 9, 6]
+
+
+@settings(max_examples=150, deadline=None)
+@given(st.lists(st.tuples(st.integers(-2**40, 2**40), st.integers(-20, 20)), min_size=1, max_size=40))
+def test_bitshift_equals_numpy_shifts(pairs):
+    """BitShift (Table 2 arithmetic): x << k for k >= 0, arithmetic
+    x >> -k for k < 0 -- numpy's left_shift / right_shift on int64 (the
+    operands are small enough that no bit leaves 64 bits)."""
+    x = np.array([a for a, _ in pairs], dtype=np.int64)
+    k = np.array([b for _, b in pairs], dtype=np.int64)
+    p = oracle.run("s := BitShift(x, k)", x=x, k=k)
+    exp = np.where(k >= 0, np.left_shift(x, np.maximum(k, 0)), np.right_shift(x, np.maximum(-k, 0)))
+    assert p.get("s") == exp.tolist()
+    # the BitShift by a constant of the Fig 3 / A15 composite key: x*2^b
+    p = oracle.run("s := BitShift(x, 3)", x=x)
+    assert p.get("s") == (x * 8).tolist()
+
+
+@settings(max_examples=150, deadline=None)
+@given(st.lists(st.tuples(st.integers(0, 3), st.integers(-1000, 1000), st.booleans()), min_size=1, max_size=60))
+def test_foldscan_equals_pandas_cumsum_of_runs_with_epsilon(triples):
+    """FoldScan (reading A27): per adjacency run, the inclusive
+    cumulative sum of the non-epsilon values (pandas groupby.cumsum over the
+    runs with epsilon as 0); an epsilon slot stays epsilon."""
+    ctrl = np.array([c for c, _, _ in triples])
+    val = np.array([v for _, v, _ in triples])
+    eps = np.array([e for _, _, e in triples])
+    p = oracle.run("s := FoldScan(c, v)", c=ctrl, v=(val, eps))
+    rid = _runs_by_adjacency(ctrl)
+    cs = pd.Series(np.where(eps, 0, val)).groupby(rid).cumsum().to_numpy()
+    exp = [None if e else int(x) for x, e in zip(cs, eps)]
+    assert p.get("s") == exp

@@ -188,3 +188,91 @@ def test_q15_interpreter_bruteforce_pandas(sf):
     keys = [k for k in p.get("o_key") if k is not None]
     got = {k + kmin: (p.get("o_rev")[j], p.get("o_cnt")[j]) for j, k in enumerate(keys)}
     assert got == bf
+
+
+def _q1_with_eps_bruteforce(li, eps, ship_max=10471):
+    """Q1 over epsilon-laden rows by plain Python loops, from the rules
+    alone: a term over epsilon is false (A9), an epsilon key code gives the
+    row no group, an epsilon operand makes a product epsilon and a SUM skips
+    epsilon values (A5); COUNT(*) counts the group's rows."""
+    acc = {}
+    n = len(li["l_shipdate"])
+    for i in range(n):
+        if eps["l_shipdate"][i] or not li["l_shipdate"][i] <= ship_max:
+            continue
+        if eps["l_returnflag"][i] or eps["l_linestatus"][i]:
+            continue
+        k = int(li["l_returnflag"][i]) * 2 + int(li["l_linestatus"][i])
+        a = acc.setdefault(k, [0] * 6)
+        q, e, d, t = (None if eps[c][i] else int(li[c][i]) for c in ("l_quantity", "l_extendedprice",
+                                                                     "l_discount", "l_tax"))
+        if q is not None:
+            a[0] += q
+        if e is not None:
+            a[1] += e
+        if e is not None and d is not None:
+            a[2] += e * (100 - d)
+            if t is not None:
+                a[3] += e * (100 - d) * (100 + t)
+        if d is not None:
+            a[4] += d
+        a[5] += 1
+    return acc
+
+
+@pytest.mark.parametrize("frac", [0.0, 0.05, 0.5])
+def test_q1_program_with_epsilon_equals_rule_loop(frac):
+    """Pins the interpreter's Q1 program (programs.Q1 + COUNT(*) = FoldCount
+    over the scattered key) on epsilon-laden input -- the expected values the
+    GPU epsilon tests take from it -- against a loop over the A5/A9 rules."""
+    n = 3000
+    li = {k: gen.host(c, n, sf=0.01) for k, c in gen.LINEITEM_COLS.items()}
+    rng = np.random.default_rng(int(frac * 100) + 1)
+    cols = ["l_shipdate", "l_returnflag", "l_linestatus", "l_quantity", "l_extendedprice", "l_discount", "l_tax"]
+    eps = {c: rng.random(n) < frac for c in cols}
+    p = oracle.Program()
+    for c in cols:
+        p.set("lineitem." + c, li[c], eps[c])
+    p.run(programs.Q1.format(ship_max_p1=10472) + """
+rows := FoldCount(sc.key, sc.key)
+gpos2 := FoldSelect(rows)
+r_key := Gather(gkey, gpos2)
+r_qty := Gather(s_qty, gpos2)
+r_base := Gather(s_base, gpos2)
+r_dp := Gather(s_dp, gpos2)
+r_ch := Gather(s_ch, gpos2)
+r_disc := Gather(s_disc, gpos2)
+r_rows := Gather(rows, gpos2)
+""")
+    outs = [p.get(o) for o in ("r_qty", "r_base", "r_dp", "r_ch", "r_disc", "r_rows")]
+    got = {k: [(o[j] or 0) for o in outs] for j, k in enumerate(p.get("r_key")) if k is not None}
+    assert got == _q1_with_eps_bruteforce(li, eps)
+    if frac == 0.0:
+        assert got == oracle.q1(li)
+
+
+@pytest.mark.parametrize("frac", [0.0, 0.05, 0.5])
+def test_q6_program_with_epsilon_equals_rule_loop(frac):
+    """The same pin for programs.Q6 with COUNT(*) = FoldSum of FoldCount(fold,
+    positions): a row qualifies only if every term is non-epsilon and true;
+    an epsilon l_extendedprice makes the product epsilon (skipped)."""
+    n = 5000
+    li = {k: gen.host(c, n, sf=0.01) for k, c in gen.LINEITEM_COLS.items()}
+    # widen the window so that many rows qualify
+    rng = np.random.default_rng(int(frac * 100) + 2)
+    cols = ["l_shipdate", "l_discount", "l_quantity", "l_extendedprice"]
+    eps = {c: rng.random(n) < frac for c in cols}
+    p = oracle.Program()
+    for c in cols:
+        p.set("lineitem." + c, li[c], eps[c])
+    p.run(programs.Q6.format(intent=97, d0m1=8000, d1=10000, dlom1=2, dhip1=9, qmax=4000)
+          + "pc2 := FoldCount(fold, positions)\ncount2 := FoldSum(pc2)\n")
+    rev = cnt = 0
+    for i in range(n):
+        if any(eps[c][i] for c in ("l_shipdate", "l_discount", "l_quantity")):
+            continue
+        if 8001 <= li["l_shipdate"][i] < 10000 and 3 <= li["l_discount"][i] <= 8 and li["l_quantity"][i] < 4000:
+            cnt += 1
+            if not eps["l_extendedprice"][i]:
+                rev += int(li["l_extendedprice"][i]) * int(li["l_discount"][i])
+    assert (p.get("revenue")[0] or 0, p.get("count2")[0]) == (rev, cnt)
