@@ -445,6 +445,50 @@ vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const v
                         const vd_agg* aggs, int32_t naggs, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
                         int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
 
+/* Grouped fold over SPARSE keys: when the key domain
+ * max - min + 1 is far larger than the number of distinct keys (64-bit
+ * surrogate or hashed keys), identity hashing over min..max (vd_group_fold,
+ * P:L1054-1056) cannot size its table.  Here the open-addressing table is
+ * sized from `max_groups`, an upper bound on the distinct qualifying keys
+ * (capacity: the power of two >= 2 x max_groups), and keys are placed by a
+ * 64-bit mixing hash with linear probing: each CTA folds into a private
+ * shared-memory table first and SPILLS to the global table (workspace,
+ * global reductions) when a key finds no free slot there; the CTA's table
+ * is flushed into the global one at its end.  Then the FoldSelect
+ * compaction of the occupied slots (Fig 11).
+ *   cols, n, pred, key_col (i32/i64, no metadata needed), aggs : as
+ *       vd_group_fold (integer SUMs proven int64-exact from min/max x n, else
+ *       VD_E_OVERFLOW; float SUM f64 in an unspecified order; integer MIN /
+ *       MAX; epsilon keys have no group; epsilon factors are skipped).
+ *   outputs: as vd_group_fold, but the groups come in TABLE order (a hash
+ *       table has no key order; vd_group_fold is the ascending-key variant).
+ *       *out_ngroups_dev = -1 if more than the capacity's distinct keys
+ *       arrived (the table filled up; results are then incomplete).
+ *   ws : vd_hash_group_fold_ws_bytes(max_groups, naggs) bytes. */
+#define VD_MAX_HASH_GROUPS ((int64_t)1 << 28)
+vd_status vd_hash_group_fold_ws_bytes(int64_t max_groups, int32_t naggs, size_t* bytes_host);
+vd_status vd_hash_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const vd_pred* pred, int32_t key_col,
+                             const vd_agg* aggs, int32_t naggs, int64_t max_groups, int64_t* out_keys, void* out_aggs,
+                             int64_t* out_rows, int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
+
+/* Cross-GPU merge of COMPACTED groups (the Fig 3 hierarchical fold one
+ * level above GPUs, for high-cardinality grouping): `ngroups`
+ * (host count) groups -- e.g. every rank's vd_group_fold / vd_hash_group_fold
+ * output, concatenated after an all-gather -- are re-inserted into one hash
+ * table: equal keys combine (integer SUM / COUNT exactly in 128 bits, float
+ * SUM in f64 in an unspecified order, MIN / MAX over the non-epsilon
+ * values, row counts added) and the result is compacted in table order.
+ *   keys / aggs / rows : device, the vd_group_fold output layout (16-byte
+ *       aggregate slots, naggs per group).
+ *   kinds_host[a] / isf_host[a] : aggregate kind and whether it is f64.
+ *   max_groups : bound on the distinct keys; *out_ngroups_dev = -1 if exceeded.
+ *   ws : vd_merge_groups_ws_bytes(max_groups, naggs). */
+vd_status vd_merge_groups_ws_bytes(int64_t max_groups, int32_t naggs, size_t* bytes_host);
+vd_status vd_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, int64_t ngroups,
+                          const int32_t* kinds_host, const int32_t* isf_host, int32_t naggs, int64_t max_groups,
+                          int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ngroups_dev, void* ws,
+                          size_t ws_bytes, void* stream);
+
 /* Compacted result of a pipeline: the FoldSelect compaction of Fig 11
  * applied to the merged partials -- the non-empty groups
  * (row count > 0), in ascending key order (reading A16), empty groups

@@ -675,6 +675,44 @@ vd_status vd_group_fold_ws_bytes(int64_t domain, int32_t naggs, size_t* bytes) {
     return VD_OK;
 }
 
+// Aggregates of a grouped fold over int64 table words (vd_group_fold,
+// vd_hash_group_fold): factor columns in range, float aggregates SUM only,
+// integer SUMs provably exact in int64 over all n rows (min/max metadata).
+static vd_status check_group_aggs(const vd_column* cols, int32_t ncols, int64_t n, const vd_agg* aggs, int32_t naggs,
+                                  int32_t* isf, const char* tag) {
+    for (int a = 0; a < naggs; ++a) {
+        const vd_agg& g = aggs[a];
+        if (g.kind < VD_AGG_SUM || g.kind > VD_AGG_MAX) { set_error("bad aggregate kind"); return VD_E_ARG; }
+        if (g.kind == VD_AGG_COUNT) continue;
+        if (g.nfactors < 1 || g.nfactors > VD_MAX_FACTORS) { set_error("nfactors in [1, 3]"); return VD_E_ARG; }
+        double mx = 1.0;  // bound of |product|
+        bool known = true;
+        for (int f = 0; f < g.nfactors; ++f) {
+            const vd_factor& fc = g.f[f];
+            if (fc.col < -1 || fc.col >= ncols) { set_error("factor column out of range"); return VD_E_ARG; }
+            if (fc.col < 0) { mx *= std::fabs((double)fc.a); continue; }
+            const vd_column& c = cols[fc.col];
+            if (c.dtype == VD_F32 || c.dtype == VD_F64) { isf[a] = 1; continue; }
+            if (!c.has_minmax) { known = false; continue; }
+            const double x1 = (double)fc.a + (double)fc.b * (double)c.min, x2 = (double)fc.a + (double)fc.b * (double)c.max;
+            mx *= std::max(std::fabs(x1), std::fabs(x2));
+        }
+        if (isf[a] && g.kind != VD_AGG_SUM) {
+            set_error(std::string(tag) + ": float MIN/MAX not supported");
+            return VD_E_UNSUPPORTED;
+        }
+        if (isf[a]) continue;
+        // int64 table slots: a SUM must be exact over all n rows, MIN/MAX must
+        // stay below the table's identity values
+        const double lim = g.kind == VD_AGG_SUM ? mx * (double)(n > 0 ? n : 1) : mx;
+        if (!known || lim >= 9.2e18) {
+            set_error(std::string(tag) + ": min/max metadata cannot prove int64 aggregates exact");
+            return VD_E_OVERFLOW;
+        }
+    }
+    return VD_OK;
+}
+
 vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const vd_pred* pred, int32_t key_col,
                         const vd_agg* aggs, int32_t naggs, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
                         int64_t* out_ngroups, void* ws, size_t ws_bytes, void* stream) {
@@ -702,33 +740,7 @@ vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const v
     if (kc.max < kc.min || dspan > (double)VD_MAX_DOMAIN) { set_error("group_fold: key domain exceeds VD_MAX_DOMAIN"); return VD_E_DOMAIN; }
     const int64_t D = kc.max - kc.min + 1;
     int32_t isf[VD_MAX_AGGS] = {0};
-    for (int a = 0; a < naggs; ++a) {
-        const vd_agg& g = aggs[a];
-        if (g.kind < VD_AGG_SUM || g.kind > VD_AGG_MAX) { set_error("bad aggregate kind"); return VD_E_ARG; }
-        if (g.kind == VD_AGG_COUNT) continue;
-        if (g.nfactors < 1 || g.nfactors > VD_MAX_FACTORS) { set_error("nfactors in [1, 3]"); return VD_E_ARG; }
-        double mx = 1.0;  // bound of |product|
-        bool known = true;
-        for (int f = 0; f < g.nfactors; ++f) {
-            const vd_factor& fc = g.f[f];
-            if (fc.col < -1 || fc.col >= ncols) { set_error("factor column out of range"); return VD_E_ARG; }
-            if (fc.col < 0) { mx *= std::fabs((double)fc.a); continue; }
-            const vd_column& c = cols[fc.col];
-            if (c.dtype == VD_F32 || c.dtype == VD_F64) { isf[a] = 1; continue; }
-            if (!c.has_minmax) { known = false; continue; }
-            const double x1 = (double)fc.a + (double)fc.b * (double)c.min, x2 = (double)fc.a + (double)fc.b * (double)c.max;
-            mx *= std::max(std::fabs(x1), std::fabs(x2));
-        }
-        if (isf[a] && g.kind != VD_AGG_SUM) { set_error("group_fold: float MIN/MAX not supported"); return VD_E_UNSUPPORTED; }
-        if (isf[a]) continue;
-        // int64 table slots: a SUM must be exact over all n rows, MIN/MAX must
-        // stay below the table's identity values
-        const double lim = g.kind == VD_AGG_SUM ? mx * (double)(n > 0 ? n : 1) : mx;
-        if (!known || lim >= 9.2e18) {
-            set_error("group_fold: min/max metadata cannot prove int64 aggregates exact");
-            return VD_E_OVERFLOW;
-        }
-    }
+    if ((st = check_group_aggs(cols, ncols, n, aggs, naggs, isf, "group_fold")) != VD_OK) return st;
     if ((st = check_ws(ws, ws_bytes, group_ws_bytes(D, naggs))) != VD_OK) return st;
     if ((st = check_device()) != VD_OK) return st;
     DevPred dp;
@@ -736,6 +748,86 @@ vd_status vd_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const v
     int nl = 0;
     st = cuda_status(launch_group_fold(dc, dp, n, key_col, kc.min, D, aggs, isf, naggs, out_keys, out_aggs, out_rows,
                                        out_ngroups, ws, (cudaStream_t)stream, &nl));
+    count_launches(nl);
+    return st;
+}
+
+// ---- NEXT-4: grouped fold over sparse keys (k_hash.cu) ------------------------
+vd_status vd_hash_group_fold_ws_bytes(int64_t max_groups, int32_t naggs, size_t* bytes) {
+    if (!bytes) return VD_E_NULL;
+    if (max_groups < 1 || max_groups > VD_MAX_HASH_GROUPS || naggs < 0 || naggs > VD_MAX_AGGS) return VD_E_ARG;
+    *bytes = hash_group_ws_bytes(max_groups, naggs, false);
+    return VD_OK;
+}
+
+vd_status vd_hash_group_fold(const vd_column* cols, int32_t ncols, int64_t n, const vd_pred* pred, int32_t key_col,
+                             const vd_agg* aggs, int32_t naggs, int64_t max_groups, int64_t* out_keys, void* out_aggs,
+                             int64_t* out_rows, int64_t* out_ngroups, void* ws, size_t ws_bytes, void* stream) {
+    reset_launches();
+    if (n < 0) return VD_E_SHAPE;
+    if (ncols < 1 || ncols > VD_MAX_DEVCOLS || !cols) { set_error("hash_group_fold: columns"); return VD_E_ARG; }
+    if (naggs < 0 || naggs > VD_MAX_AGGS || (naggs > 0 && !aggs)) { set_error("hash_group_fold: naggs in [0, 8]"); return VD_E_ARG; }
+    if (max_groups < 1 || max_groups > VD_MAX_HASH_GROUPS) { set_error("hash_group_fold: max_groups"); return VD_E_ARG; }
+    if (!out_keys || !out_rows || !out_ngroups || (naggs > 0 && !out_aggs)) { set_error("hash_group_fold: outputs"); return VD_E_NULL; }
+    vd_status st;
+    DevCols dc;
+    std::memset(&dc, 0, sizeof(dc));
+    dc.ncols = ncols;
+    for (int c = 0; c < ncols; ++c) {
+        if ((st = check_col(&cols[c], n, "hash_group_fold")) != VD_OK) return st;
+        dc.p[c] = cols[c].data;
+        dc.dt[c] = cols[c].dtype;
+    }
+    if ((st = check_pred(pred, dc.dt, ncols)) != VD_OK) return st;
+    if (key_col < 0 || key_col >= ncols) { set_error("hash_group_fold: key column out of range"); return VD_E_ARG; }
+    if (cols[key_col].dtype != VD_I32 && cols[key_col].dtype != VD_I64) {
+        set_error("hash_group_fold: key must be i32/i64");
+        return VD_E_DTYPE;
+    }
+    int32_t isf[VD_MAX_AGGS] = {0};
+    if ((st = check_group_aggs(cols, ncols, n, aggs, naggs, isf, "hash_group_fold")) != VD_OK) return st;
+    if ((st = check_ws(ws, ws_bytes, hash_group_ws_bytes(max_groups, naggs, false))) != VD_OK) return st;
+    if ((st = check_device()) != VD_OK) return st;
+    DevPred dp;
+    make_devpred(pred, &dp);
+    int nl = 0;
+    st = cuda_status(launch_hash_group_fold(dc, dp, n, key_col, aggs, isf, naggs, max_groups, out_keys, out_aggs,
+                                            out_rows, out_ngroups, ws, (cudaStream_t)stream, &nl));
+    count_launches(nl);
+    return st;
+}
+
+vd_status vd_merge_groups_ws_bytes(int64_t max_groups, int32_t naggs, size_t* bytes) {
+    if (!bytes) return VD_E_NULL;
+    if (max_groups < 1 || max_groups > VD_MAX_HASH_GROUPS || naggs < 0 || naggs > VD_MAX_AGGS) return VD_E_ARG;
+    *bytes = hash_group_ws_bytes(max_groups, naggs, true);
+    return VD_OK;
+}
+
+vd_status vd_merge_groups(const int64_t* keys, const void* aggs_in, const int64_t* rows, int64_t ngroups,
+                          const int32_t* kinds_host, const int32_t* isf_host, int32_t naggs, int64_t max_groups,
+                          int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ngroups, void* ws,
+                          size_t ws_bytes, void* stream) {
+    reset_launches();
+    if (ngroups < 0) return VD_E_SHAPE;
+    if (naggs < 0 || naggs > VD_MAX_AGGS || (naggs > 0 && (!kinds_host || !isf_host))) return VD_E_ARG;
+    if (max_groups < 1 || max_groups > VD_MAX_HASH_GROUPS) { set_error("merge_groups: max_groups"); return VD_E_ARG; }
+    if ((ngroups > 0 && (!keys || !rows || (naggs > 0 && !aggs_in))) || !out_keys || !out_rows || !out_ngroups ||
+        (naggs > 0 && !out_aggs))
+        return VD_E_NULL;
+    for (int a = 0; a < naggs; ++a) {
+        if (kinds_host[a] < VD_AGG_SUM || kinds_host[a] > VD_AGG_MAX) { set_error("bad aggregate kind"); return VD_E_ARG; }
+        if (isf_host[a] && kinds_host[a] != VD_AGG_SUM && kinds_host[a] != VD_AGG_COUNT) {
+            set_error("merge_groups: float MIN/MAX not supported");
+            return VD_E_UNSUPPORTED;
+        }
+    }
+    vd_status st;
+    if ((st = check_ws(ws, ws_bytes, hash_group_ws_bytes(max_groups, naggs, true))) != VD_OK) return st;
+    if ((st = check_device()) != VD_OK) return st;
+    int nl = 0;
+    st = cuda_status(launch_merge_groups(keys, aggs_in, rows, ngroups, kinds_host, isf_host, naggs, max_groups,
+                                         out_keys, out_aggs, out_rows, out_ngroups, ws, (cudaStream_t)stream, &nl));
     count_launches(nl);
     return st;
 }

@@ -111,6 +111,17 @@ cudaError_t launch_group_fold(const DevCols& cols, const DevPred& pred, int64_t 
 cudaError_t launch_merge_partials(const vd_pipeline* plan, const int32_t* isf, const void* parts, int nparts,
                                   const vd_result& out, cudaStream_t s, int* nl);
 
+// k_hash.cu (NEXT-4, sparse keys)
+size_t hash_group_ws_bytes(int64_t max_groups, int naggs, bool wide);
+cudaError_t launch_hash_group_fold(const DevCols& cols, const DevPred& pred, int64_t n, int key_col,
+                                   const vd_agg* aggs, const int32_t* isf, int naggs, int64_t max_groups,
+                                   int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws,
+                                   cudaStream_t s, int* nl);
+cudaError_t launch_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, int64_t m,
+                                const int32_t* kinds, const int32_t* isf, int naggs, int64_t max_groups,
+                                int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws,
+                                cudaStream_t s, int* nl);
+
 int num_sms();
 
 }  // namespace vd

@@ -24,7 +24,8 @@ def test_header_declares_the_north_star_calls():
     names = declared_functions()
     for want in ["vd_load_column", "vd_select_branch", "vd_select_predicated", "vd_gather", "vd_scatter",
                  "vd_fold_sum", "vd_fold_count", "vd_fold_min", "vd_fold_max", "vd_fold_select", "vd_run_pipeline",
-                 "vd_merge_partials", "vd_merge_partials_device", "vd_workspace_bytes", "vd_partition"]:
+                 "vd_merge_partials", "vd_merge_partials_device", "vd_workspace_bytes", "vd_partition",
+                 "vd_hash_group_fold", "vd_merge_groups"]:
         assert want in names
 
 
