@@ -499,61 +499,43 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
     }
 }
 
-// ---- fused single-pass selection (TMA ring + decoupled look-back) -------------
-// One pass, no materialised predicate.  Warp roles of a CTA (one per SM):
-//   producer  : claims tiles of SF_CW x 1024 rows IN ORDER from a global
-//               counter (every predecessor of a claimed tile is claimed by a
-//               running CTA: forward progress) and streams them into an
-//               SF_STAGES-deep mbarrier ring with 1D bulk copies;
-//   consumers : warp w turns its 1024 rows of tile i into 32 ballots (bit L
-//               of ballot 4q+j <-> row q*128 + 32j + L: each ballot is a
-//               row-ordered 32-bit word), releases the ring slot, publishes
-//               its count -- and only then writes the positions of tile i-1,
-//               whose offset the look-back warp has resolved meanwhile;
-//   look-back : sums tile i's warp counts, publishes the tile aggregate at
-//               once and runs the decoupled look-back (single-pass scan over
-//               per-tile status words) for the tile's global offset.
-// Counting never waits for a look-back, so every claimed tile publishes its
-// aggregate as soon as its data lands and the inclusive-prefix frontier
-// trails the newest tile by about one L2 round trip of tiles -- within one
-// 128-tile look-back window (a coupled design, where a warp counts tile i+1
-// only after tile i's offset is known, let unpublished claimed tiles stall
-// every successor's look-back: 7.6-8.1 ms for 1e9 rows).
-// Positions: branching -- qualifying lanes store at their rank; predicated --
-// cursor arithmetic, every row stored at the cursor and the cursor advanced
-// by the predicate; then the ascending run streams out with
-// 16-byte stores.  Replaces the 3-launch bitmap path for single interval
-// terms on 4-byte columns.
-constexpr int SF_CW = 16;
-constexpr int SF_THREADS = SF_CW * 32 + 64;   // + producer warp + look-back warp
-constexpr int SF_STAGES = 2;
-constexpr int SF_ROWS = SF_CW * 1024;         // rows per tile
-constexpr int SF_STG = 1024 + 128 + 8;        // per-warp position stage (ints)
-
-struct SfShared {
-    uint64_t full[SF_STAGES], empty[SF_STAGES];
-    uint64_t cnt_bar[2], base_bar[2];
-    int64_t s_tile[SF_STAGES];
-    int64_t lb_tile[2];
-    int64_t base[2];
-    int cnt[2][SF_CW];
-    int woff[2][SF_CW];
-    uint32_t bal[2][SF_CW][32];
-};
+// ---- single-launch selection: stream + grid barrier + decode ------------------
+// One cooperative persistent kernel (one CTA per SM, all co-resident), each
+// CTA owning a contiguous range of 1024-row chunks:
+//   phase 1  a producer warp streams the CTA's rows through an SC_STAGES-deep
+//            TMA ring; consumer warp w turns 1024 rows into 32 ballots (bit L
+//            of ballot 32q'+j... each ballot is a row-ordered 32-bit word: bit
+//            L <-> row 32k + L of the chunk) and stores them as the chunk's
+//            32 bitmap words (the predicate materialised, Fig 8's break: n/8
+//            bytes, largely L2-resident) while counting; the CTA's count goes
+//            to counts[cta].
+//   barrier  one grid-wide barrier; the CTA's output base is the sum of the
+//            counts of the CTAs before it (148 values: no scan launch, no
+//            per-tile look-back chain).
+//   phase 2  the CTA decodes its bitmap in order with a running offset: per
+//            tile of SC_CW chunks, warp counts -> CTA prefix -> every warp
+//            stages its positions in shared memory (branching: qualifying
+//            lanes at their rank; predicated: cursor arithmetic, every row
+//            stored at the cursor, the cursor advanced by the predicate,
+//            P:L101-108) and streams the ascending run out with 16-byte
+//            stores.  The ring's shared memory is reused for the stages.
+// Replaces the 4-launch bitmap path (flag pass, scan, total, position pass):
+// the step pays the column read once, the bitmap's n/8 bytes twice (mostly
+// in L2) and the positions once.  A single-pass decoupled look-back variant
+// (a look-back per 64 KB tile) was measured at 5.8 ms for 1e9 rows: under a
+// full HBM stream one look-back costs several microseconds of L2 round trips,
+// far above a CTA's ~1.5 us per tile.
+static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
+constexpr int SC_CW = 16;
+constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
+constexpr int SC_STAGES = 3;
+constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
+constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
 
 template <int MODE>
-__device__ __forceinline__ void sf_write_positions(const uint32_t* __restrict__ bal, int64_t row_w, int64_t g0,
-                                                   int32_t* __restrict__ out, int32_t* __restrict__ sw, int lane,
-                                                   unsigned lt) {
-    uint32_t bw[32];
-#pragma unroll
-    for (int k = 0; k < 32; k += 4) {
-        const uint4 x = *reinterpret_cast<const uint4*>(bal + k);  // broadcast
-        bw[k] = x.x; bw[k + 1] = x.y; bw[k + 2] = x.z; bw[k + 3] = x.w;
-    }
-    // stage index a + k <-> output g0 + k, a = the output's misalignment in
-    // words, so stage groups of 4 are 16-byte output groups
-    const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+__device__ __forceinline__ int sc_stage_positions(const uint32_t (&bw)[32], int64_t row0, int a, int32_t* sw,
+                                                  int lane, unsigned lt) {
+    // stage index a + k <-> output k of the chunk
     int cur = a;
 #pragma unroll
     for (int q = 0; q < 8; ++q) {
@@ -564,7 +546,7 @@ __device__ __forceinline__ void sf_write_positions(const uint32_t* __restrict__ 
             const uint32_t w = bw[4 * q + j];
             const int f = (w >> lane) & 1u;
             const int r = __popc(w & lt);
-            const int32_t row = (int32_t)(row_w + q * 128 + j * 32 + lane);
+            const int32_t row = (int32_t)(row0 + (4 * q + j) * 32 + lane);
             if (MODE == 0) {
                 if (f) sw[pre + r] = row;
             } else {
@@ -578,10 +560,11 @@ __device__ __forceinline__ void sf_write_positions(const uint32_t* __restrict__ 
         }
         cur += cq;
     }
-    __syncwarp();
-    const int total = cur - a;
+    return cur - a;
+}
+
+__device__ __forceinline__ void sc_flush(const int32_t* sw, int a, int total, int32_t* __restrict__ ob, int lane) {
     const int ngr = (a + total + 3) >> 2;
-    int32_t* ob = out + g0 - a;  // 16-byte aligned
     for (int v = lane; v < ngr; v += 32) {
         const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
         if (4 * v >= a && 4 * v + 4 <= a + total) {
@@ -595,179 +578,201 @@ __device__ __forceinline__ void sf_write_positions(const uint32_t* __restrict__ 
             }
         }
     }
-    __syncwarp();
 }
 
 template <int MODE, typename T>
-__global__ void __launch_bounds__(SF_THREADS, 1) k_sel_fused(const T* __restrict__ col, T lo, T hi, int64_t n,
-                                                             int64_t ntiles, int32_t* __restrict__ out,
-                                                             int64_t* __restrict__ out_count,
-                                                             uint64_t* __restrict__ status,
-                                                             unsigned long long* __restrict__ tile_ctr) {
-    constexpr uint32_t TB = SF_ROWS * sizeof(T);
+__global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
+                                                            int32_t* __restrict__ out, int64_t* __restrict__ out_count,
+                                                            uint32_t* __restrict__ bits,
+                                                            int64_t* __restrict__ counts,
+                                                            unsigned int* __restrict__ grid_bar) {
+    constexpr uint32_t TB = SC_CHUNKS * 1024 * sizeof(T);  // tile bytes
     extern __shared__ __align__(128) uint8_t smem[];
-    int32_t* stage = reinterpret_cast<int32_t*>(smem + (size_t)SF_STAGES * TB);
-    SfShared& S = *reinterpret_cast<SfShared*>(stage + SF_CW * SF_STG);
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)SC_STAGES * TB);
+    uint64_t* empty = full + SC_STAGES;
+    __shared__ int s_cnt[SC_CW];
+    __shared__ int64_t s_base;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int64_t nfull = n / SF_ROWS;  // tiles loaded by TMA; the ragged last one by LDG
+    // the CTA's chunk range [c0, c1) (chunk = 1024 rows), tiles of SC_CHUNKS
+    const int64_t nchunks = (n + 1023) / 1024;
+    const int64_t c0 = nchunks * blockIdx.x / gridDim.x, c1 = nchunks * (blockIdx.x + 1) / gridDim.x;
+    const int64_t ntile = (c1 - c0 + SC_CHUNKS - 1) / SC_CHUNKS;
     if (threadIdx.x == 0) {
-        for (int i = 0; i < SF_STAGES; ++i) {
-            mbar_init(&S.full[i], 1);
-            mbar_init(&S.empty[i], SF_CW);
-        }
-        for (int i = 0; i < 2; ++i) {
-            mbar_init(&S.cnt_bar[i], SF_CW);
-            mbar_init(&S.base_bar[i], 1);
+        for (int i = 0; i < SC_STAGES; ++i) {
+            mbar_init(&full[i], 1);
+            mbar_init(&empty[i], SC_CW);
         }
         fence_mbar_init();
     }
     __syncthreads();
-    if (warp == SF_CW) {
-        // ---- producer: claim tiles in order, stream them into the ring ----
+    // ---- phase 1: stream -> ballot words + count ----
+    int64_t cnt = 0;
+    if (warp == SC_CW) {
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
             int st = 0;
             uint32_t ph = 0;
-            for (int64_t it = 0;; ++it) {
-                if (it >= SF_STAGES) mbar_wait(&S.empty[st], ph ^ 1u);
-                const int64_t tile = (int64_t)atomicAdd(tile_ctr, 1ull);
-                if (tile >= ntiles) {
-                    S.s_tile[st] = -1;
-                    mbar_arrive(&S.full[st]);
-                    break;
-                }
-                S.s_tile[st] = tile;
-                if (tile < nfull) {
-                    mbar_expect_tx(&S.full[st], TB);
-                    tma_load_1d(smem + (size_t)st * TB, col + tile * SF_ROWS, TB, &S.full[st], pol);
+            for (int64_t t = 0; t < ntile; ++t) {
+                if (t >= SC_STAGES) mbar_wait(&empty[st], ph ^ 1u);
+                const int64_t r0 = (c0 + t * SC_CHUNKS) * 1024;
+                const int64_t r1 = min((c0 + (t + 1) * SC_CHUNKS) * 1024, c1 * 1024);
+                if (r1 <= n && ((r1 - r0) * (int64_t)sizeof(T)) % 16 == 0) {
+                    const uint32_t bytes = (uint32_t)((r1 - r0) * sizeof(T));
+                    mbar_expect_tx(&full[st], bytes);
+                    tma_load_1d(smem + (size_t)st * TB, col + r0, bytes, &full[st], pol);
                 } else {
-                    mbar_arrive(&S.full[st]);  // partial tile: the consumers read it from global memory
+                    mbar_arrive(&full[st]);  // the ragged end of the column: consumers load it directly
                 }
-                if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
+                if (++st == SC_STAGES) { st = 0; ph ^= 1u; }
             }
-        }
-        return;
-    }
-    if (warp == SF_CW + 1) {
-        // ---- look-back: tile aggregate -> published -> global offset ----
-        for (int64_t i = 0;; ++i) {
-            const int sl = (int)(i & 1);
-            mbar_wait(&S.cnt_bar[sl], (uint32_t)((i >> 1) & 1));
-            const int64_t tile = S.lb_tile[sl];
-            if (tile < 0) break;
-            const int v = lane < SF_CW ? S.cnt[sl][lane] : 0;
-            int incl = v;
-#pragma unroll
-            for (int o = 1; o < SF_CW; o <<= 1) {
-                const int u = __shfl_up_sync(VD_FULL, incl, o);
-                if (lane >= o) incl += u;
-            }
-            if (lane < SF_CW) S.woff[sl][lane] = incl - v;
-            const int64_t agg = __shfl_sync(VD_FULL, incl, SF_CW - 1);
-            const int64_t base = lookback_exclusive_w128(status, tile, agg, lane);
-            if (lane == 0) {
-                S.base[sl] = base;
-                if (tile == ntiles - 1) *out_count = base + agg;
-                mbar_arrive(&S.base_bar[sl]);
-            }
-            __syncwarp();
-        }
-        return;
-    }
-    // ---- consumers ----
-    const unsigned lt = lanemask_lt();
-    int32_t* sw = stage + warp * SF_STG;
-    int st = 0;
-    uint32_t ph = 0;
-    int64_t prev_tile = -1;
-    for (int64_t i = 0;; ++i) {
-        const int sl = (int)(i & 1);
-        mbar_wait(&S.full[st], ph);
-        const int64_t tile = S.s_tile[st];
-        if (tile >= 0) {
-            const int64_t row_w = tile * SF_ROWS + (int64_t)warp * 1024;
-            uint32_t* mybal = S.bal[sl][warp];
-            int cnt = 0;
-            if (tile < nfull) {
-                const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
-#pragma unroll
-                for (int k = 0; k < 32; ++k) {
-                    const T v = src[k * 32 + lane];
-                    const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN (epsilon) fails
-                    if (lane == k) mybal[k] = b;
-                    cnt += __popc(b);
-                }
-            } else {
-#pragma unroll
-                for (int k = 0; k < 32; ++k) {
-                    const int64_t r = row_w + k * 32 + lane;
-                    bool f = false;
-                    if (r < n) {
-                        const T v = __ldg(col + r);
-                        f = v >= lo && v <= hi;
-                    }
-                    const uint32_t b = __ballot_sync(VD_FULL, f);
-                    if (lane == k) mybal[k] = b;
-                    cnt += __popc(b);
-                }
-            }
-            __syncwarp();
-            if (lane == 0) {
-                mbar_arrive(&S.empty[st]);  // slot free: only the ballots are needed from here
-                S.cnt[sl][warp] = cnt;
-                if (warp == 0) S.lb_tile[sl] = tile;
-            }
-        } else if (warp == 0 && lane == 0) {
-            S.lb_tile[sl] = -1;  // tells the look-back warp to stop
         }
         __syncwarp();
-        if (lane == 0) mbar_arrive(&S.cnt_bar[sl]);
-        if (++st == SF_STAGES) { st = 0; ph ^= 1u; }
-        // positions of the previous tile, whose offset is resolved by now
-        if (prev_tile >= 0) {
-            const int ps = sl ^ 1;
-            mbar_wait(&S.base_bar[ps], (uint32_t)(((i - 1) >> 1) & 1));
-            const int64_t g0 = S.base[ps] + S.woff[ps][warp];
-            sf_write_positions<MODE>(S.bal[ps][warp], prev_tile * SF_ROWS + (int64_t)warp * 1024, g0, out, sw, lane,
-                                     lt);
+    } else {
+        int st = 0;
+        uint32_t ph = 0;
+        for (int64_t t = 0; t < ntile; ++t) {
+            mbar_wait(&full[st], ph);
+            const int64_t c = c0 + t * SC_CHUNKS + warp;  // this warp's chunk
+            const int64_t r0 = (c0 + t * SC_CHUNKS) * 1024;
+            const int64_t r1 = min((c0 + (t + 1) * SC_CHUNKS) * 1024, c1 * 1024);
+            const bool staged = r1 <= n && ((r1 - r0) * (int64_t)sizeof(T)) % 16 == 0;
+            uint32_t mine = 0;
+            if (c < c1) {
+                const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
+#pragma unroll 8
+                for (int k = 0; k < 32; ++k) {
+                    const int64_t r = c * 1024 + k * 32 + lane;
+                    bool f;
+                    if (staged) {
+                        const T v = src[k * 32 + lane];
+                        f = v >= lo && v <= hi;  // NaN / INT_MIN (epsilon) fail: bounds from the host
+                    } else {
+                        f = false;
+                        if (r < n) {
+                            const T v = __ldg(col + r);
+                            f = v >= lo && v <= hi;
+                        }
+                    }
+                    const uint32_t b = __ballot_sync(VD_FULL, f);
+                    if (lane == k) mine = b;
+                }
+                bits[c * 32 + lane] = mine;
+                cnt += __popc(mine);
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&empty[st]);
+            if (++st == SC_STAGES) { st = 0; ph ^= 1u; }
         }
-        if (tile < 0) break;
-        prev_tile = tile;
+    }
+    // CTA count -> counts[cta]
+#pragma unroll
+    for (int o = 16; o; o >>= 1) cnt += __shfl_xor_sync(VD_FULL, cnt, o);
+    if (lane == 0 && warp < SC_CW) s_cnt[warp] = (int)cnt;
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        int64_t t = 0;
+        for (int w = 0; w < SC_CW; ++w) t += s_cnt[w];
+        st_release_u64(reinterpret_cast<uint64_t*>(&counts[blockIdx.x]), (uint64_t)t);
+        // ---- grid barrier (cooperative launch: every CTA is resident) ----
+        __threadfence();
+        atomicAdd(grid_bar, 1u);
+        while (ld_acquire_u32(grid_bar) < gridDim.x) __nanosleep(64);
+    }
+    __syncthreads();
+    // CTA base = counts of the CTAs before it
+    if (warp == 0) {
+        int64_t b = 0;
+        for (int i = lane; i < (int)blockIdx.x; i += 32) b += (int64_t)ld_acquire_u64(reinterpret_cast<uint64_t*>(&counts[i]));
+        b = warp_sum_i64(b);
+        if (lane == 0) {
+            s_base = b;
+            if (blockIdx.x == gridDim.x - 1) {
+                int64_t tot = b;
+                for (int w = 0; w < SC_CW; ++w) tot += s_cnt[w];
+                *out_count = tot;
+            }
+        }
+    }
+    __syncthreads();
+    // ---- phase 2: bitmap words -> positions ----
+    if (warp == SC_CW) return;
+    const unsigned lt = lanemask_lt();
+    int32_t* sw = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
+    int64_t run = s_base;
+    for (int64_t t = 0; t < ntile; ++t) {
+        const int64_t c = c0 + t * SC_CHUNKS + warp;
+        const uint32_t word = c < c1 ? __ldcs(&bits[c * 32 + lane]) : 0u;
+        const int wc = __popc(word);
+        int tot = wc;
+#pragma unroll
+        for (int o = 16; o; o >>= 1) tot += __shfl_xor_sync(VD_FULL, tot, o);
+        if (lane == 0) s_cnt[warp] = tot;
+        bar_sync_n(1, SC_CW * 32);
+        int woff = 0, ttot = 0;
+#pragma unroll
+        for (int w = 0; w < SC_CW; ++w) {
+            const int x = s_cnt[w];
+            woff += w < warp ? x : 0;
+            ttot += x;
+        }
+        bar_sync_n(1, SC_CW * 32);  // s_cnt is rewritten next tile
+        if (c < c1 && tot > 0) {
+            uint32_t bw[32];
+#pragma unroll
+            for (int k = 0; k < 32; ++k) bw[k] = __shfl_sync(VD_FULL, word, k);
+            const int64_t g0 = run + woff;
+            const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+            const int total = sc_stage_positions<MODE>(bw, c * 1024, a, sw, lane, lt);
+            __syncwarp();
+            sc_flush(sw, a, total, out + g0 - a, lane);
+            __syncwarp();
+        }
+        run += ttot;
     }
 }
 
-static size_t sel_fused_smem(size_t tsize) {
-    return (size_t)SF_STAGES * SF_ROWS * tsize + (size_t)SF_CW * SF_STG * 4 + sizeof(SfShared);
+static size_t sel_coop_smem(size_t tsize) {
+    const size_t ring = (size_t)SC_STAGES * SC_CHUNKS * 1024 * tsize + 2 * SC_STAGES * 8;
+    const size_t stg = (size_t)SC_CW * SC_STG * 4;
+    return ring > stg ? ring : stg;
 }
 
-// VD_SELECT_FUSED=0 keeps the bitmap path (comparison runs)
-static bool use_sel_fused() {
+// VD_SELECT_COOP=0 keeps the 4-launch bitmap path (comparison runs)
+static bool use_sel_coop() {
     static const bool off = [] {
-        const char* e = getenv("VD_SELECT_FUSED");
+        const char* e = getenv("VD_SELECT_COOP");
         return e && strcmp(e, "0") == 0;
     }();
     return !off;
 }
 
 template <int MODE, typename T>
-static cudaError_t run_select_fused(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
-                                    void* ws, cudaStream_t s, int* nl) {
-    const int64_t ntiles = (n + SF_ROWS - 1) / SF_ROWS;
-    if (ntiles == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
-    unsigned long long* ctr = (unsigned long long*)ws;
-    uint64_t* status = (uint64_t*)((char*)ws + 256);
-    cudaError_t e = cudaMemsetAsync(ws, 0, 256 + (size_t)ntiles * 8, s);
-    if (e != cudaSuccess) return e;
-    const size_t sm = sel_fused_smem(sizeof(T));
-    auto kern = k_sel_fused<MODE, T>;
+static cudaError_t run_select_coop(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
+                                   void* ws, cudaStream_t s, int* nl) {
+    if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
+    const int64_t nchunks = (n + 1023) / 1024;
+    char* w = (char*)ws;
+    unsigned int* bar = (unsigned int*)w;
+    int64_t* counts = (int64_t*)(w + 256);
+    uint32_t* bits = (uint32_t*)(w + 256 + al256((size_t)4096 * 8));
+    const size_t sm = sel_coop_smem(sizeof(T));
+    auto kern = k_sel_coop<MODE, T>;
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
     int per_sm = 0;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SF_THREADS, sm) != cudaSuccess || per_sm < 1)
-        per_sm = 1;
-    const int grid = (int)std::min<int64_t>(ntiles, (int64_t)num_sms() * per_sm);
-    kern<<<grid, SF_THREADS, sm, s>>>(col, lo, hi, n, ntiles, out_pos, out_count, status, ctr);
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SC_THREADS, sm) != cudaSuccess || per_sm < 1)
+        return cudaErrorCooperativeLaunchTooLarge;
+    int grid = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, std::min<int64_t>(nchunks, 4096));
+    cudaError_t e = cudaMemsetAsync(bar, 0, 4, s);
+    if (e != cudaSuccess) return e;
+    void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&out_pos, (void*)&out_count,
+                    (void*)&bits, (void*)&counts, (void*)&bar};
+    e = cudaLaunchCooperativeKernel((const void*)kern, dim3(grid), dim3(SC_THREADS), args, sm, s);
     ++*nl;
-    return cudaGetLastError();
+    return e;
+}
+static size_t sel_coop_ws_bytes(int64_t n) {
+    const int64_t nchunks = (n + 1023) / 1024;
+    return 256 + al256((size_t)4096 * 8) + al256((size_t)nchunks * 32 * 4);
 }
 
 // Per-row predicates (several columns, run heads): ballot j is word j.
@@ -898,7 +903,6 @@ struct BmLayout {
     int64_t* offs;
     void* scan_ws;
 };
-static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
 static BmLayout bm_layout(int64_t n, void* ws) {
     BmLayout L;
     L.nchunks = (n + BM_CHUNK - 1) / BM_CHUNK;
@@ -947,10 +951,10 @@ static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t*
 }
 
 size_t select_ws_bytes(int64_t n) {
-    int64_t ntiles = (n + std::min(SEL_TILE, SF_ROWS) - 1) / std::min(SEL_TILE, SF_ROWS);
+    int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
     size_t b = 256 + (size_t)ntiles * 8;
     size_t lb = (b + 255) & ~(size_t)255;
-    size_t bm = bm_ws_bytes(n);
+    size_t bm = std::max(bm_ws_bytes(n), sel_coop_ws_bytes(n));
     return lb > bm ? lb : bm;
 }
 
@@ -1043,8 +1047,8 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         if constexpr (sizeof(T) == 4) {
-            if (ivl && use_sel_fused() && ((uintptr_t)p & 15) == 0)
-                return run_select_fused<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+            if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0)
+                return run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
         }
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L) {

@@ -52,3 +52,20 @@ def test_two_ranks_merge_equals_one(workload):
         exp = oracle.q1(li)
         got = {int(k): [int(x) for x in v[:6]] for k, v in one["result"].items()}
         assert got == exp
+
+
+@pytest.mark.parametrize("workload", ["q1", "q6"])
+def test_nccl_two_gpus_merge_equals_one(workload):
+    """The production N>1 path: one rank per GPU over NCCL (all-gather of the
+    partials captured in a CUDA graph with the device merge).  gpurun boxes
+    have one GPU, so this runs only where two are visible."""
+    import torch
+    if torch.cuda.device_count() < 2:
+        pytest.skip("needs two GPUs (NCCL over NVLink)")
+    sf = 1.0
+    common = ["--workload", workload, "--sf", str(sf), "--steps", "5", "--warmup", "3", "--no-cpu-baseline",
+              "--no-e2e"]
+    one = _bench(common)
+    two = _bench(common + ["--gpus", "2"], nproc=2)
+    assert two["n_gpus"] == 2 and two["cuda_graphs"] == "pipeline + (all-gather, merge)"
+    assert two["result_digest"] == one["result_digest"]

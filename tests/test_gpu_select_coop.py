@@ -1,10 +1,11 @@
-"""The fused single-pass selection kernel (k_sel_fused: TMA ring, ballot
-words in registers, decoupled look-back, staged 16-byte stores) against the
-oracle, at sizes around its 8192-row tile (full tiles by TMA, the ragged
-last tile by LDG), all-false / all-true tiles, NaN (epsilon, never
-selected: A9), int32 columns, unaligned outputs, branching and predicated
-(identical positions), and the same inputs through the bitmap
-path (VD_SELECT_FUSED=0) it replaces."""
+"""The single-launch selection kernel (k_sel_coop: per-CTA contiguous chunk
+ranges streamed by TMA into ballot words, one grid barrier, in-order decode
+into staged 16-byte stores) against the oracle: sizes from one row to
+several 16-chunk tiles per CTA with a ragged end (TMA tiles, LDG for the
+column's last partial chunk), all-false / all-true tiles, NaN (epsilon,
+never selected: A9), int32 columns, unaligned outputs, branching and
+predicated (identical positions), and the same inputs through
+the 4-launch bitmap path (VD_SELECT_COOP=0) it replaces."""
 import numpy as np
 import pytest
 import torch
@@ -17,7 +18,7 @@ from test_gpu_pipeline import env
 
 pytestmark = pytest.mark.gpu
 
-SIZES = [1, 31, 8191, 8192, 8193, 3 * 8192 + 5, 70001, 1 << 20]
+SIZES = [1, 31, 1023, 1024, 1025, 3 * 8192 + 5, 70001, 1 << 20, 148 * 16 * 1024 * 3 + 4097]
 
 
 def _select(fn, v, n, t, shift=0):
@@ -43,7 +44,7 @@ def test_fused_select_f32_vs_oracle(mode, n, t):
     dv = torch.from_numpy(v).cuda()
     got = _select(fn, dv, n, t)
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
-    with env(VD_SELECT_FUSED="0"):  # the bitmap path agrees
+    with env(VD_SELECT_COOP="0"):  # the bitmap path agrees
         assert np.array_equal(_select(fn, dv, n, t), pos_o)
 
 
