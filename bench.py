@@ -60,12 +60,15 @@ def parse():
     ap.add_argument("--strategy", default="layout", choices=["single", "separate", "layout"],
                     help="fig14: Single Loop / Separate Loops / Layout Transform (P:L1156-1193)")
     ap.add_argument("--pattern", default="random", choices=["random", "sequential"], help="fig14 lookup pattern")
-    ap.add_argument("--target-mb", type=int, default=128, help="fig14 target table size (two int32 columns)")
+    ap.add_argument("--target-mb", type=int, default=1024, help="fig14 target table size (two int32 columns)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     ap.add_argument("--seed", type=int, default=0x5EEDC0DE)
     ap.add_argument("--no-graph", action="store_true", help="N > 1: launch eagerly instead of CUDA graphs")
+    ap.add_argument("--grouping", default="direct", choices=["direct", "hash"],
+                    help="q15: identity-hashed table over min..max (vd_group_fold) or open addressing "
+                         "(vd_hash_group_fold)")
     ap.add_argument("--dist-backend", default="nccl", choices=["nccl", "gloo"],
                     help="process-group backend for N > 1 (gloo: test mode, ranks may share a GPU)")
     return ap.parse_args()
@@ -384,12 +387,7 @@ def main():
     stream = torch.cuda.current_stream()
 
     w = args.workload
-    if w == "select":
-        n_total = args.rows or 10**9
-    elif w == "fkjsel":
-        n_total = args.rows or 200_000_000
-    else:
-        n_total = gen.lineitem_rows(sf)
+    n_total = workload_rows(args, w, sf)
     a, b = rank * n_total // world, (rank + 1) * n_total // world
     n = b - a
     sel_mode = {"branch": vd.VD_SEL_BRANCH, "predicated": vd.VD_SEL_PREDICATED,
@@ -558,8 +556,8 @@ def main():
     alg_bytes = n * bpr
     extra = {}
     if w == "fkjsel":
-        # reading A33: a lookup into a table larger than L2 (16 Mi x 8 B =
-        # 128 MiB) moves one 64-byte HBM block; branching and predicated-lookup
+        # reading A33: a lookup into a table larger than L2 (128 Mi x 8 B =
+        # 1 GiB) moves one 64-byte HBM block; branching and predicated-lookup
         # plans look up the qualifying rows only (the lookup plan sends the
         # rest to the hot slot 0), predicated aggregation looks up every row
         sel_rows = int(next(iter(result.values()))[-1]) if result else 0
@@ -718,7 +716,9 @@ def c1_main(args, rank, world, local):
     4 MiB input is L2-resident by design, so the HBM roofline does not
     apply: per-call microseconds are reported warm (back to back) and cold
     (each call after a 512 MB write that evicts L2), on the launching stream
-    with CUDA events.  A step = positions + sum, both modes reported; the
+    with CUDA events around CUDA-graph replays of each call (so the events
+    time GPU work, not Python marshalling).  A step = positions + sum, both
+    modes reported; the
     line's value is the warm branching step.  Each rank runs an independent
     replica (C1 does not shard: 'replicas only')."""
     import numpy as np
@@ -754,12 +754,34 @@ def c1_main(args, rank, world, local):
         calls = {"positions": lambda: sel(col, n, p, out_pos=pos, out_count=cnt, ws=ws, stream=stream),
                  "sum": lambda: vd.run_pipeline(plan, col, n, out=out, ws=pws, stream=stream)}
         for _ in range(max(args.warmup, 3)):
+            nl = 0
             for f in calls.values():
                 f()
+                nl += vd.last_launch_count()
+        torch.cuda.synchronize()
+        # each call captured once in a CUDA graph and replayed: the events then
+        # time the GPU work, not the Python marshalling between launches
+        graphs = {}
+        side = torch.cuda.Stream(device=dev)
+        side.wait_stream(stream)
+        for name, f in list(calls.items()) + [("step", lambda: [g() for g in calls.values()])]:
+            g = torch.cuda.CUDAGraph()
+            with torch.cuda.stream(side):
+                with torch.cuda.graph(g, stream=side):
+                    if name == "positions":
+                        sel(col, n, p, out_pos=pos, out_count=cnt, ws=ws, stream=side)
+                    elif name == "sum":
+                        vd.run_pipeline(plan, col, n, out=out, ws=pws, stream=side)
+                    else:
+                        sel(col, n, p, out_pos=pos, out_count=cnt, ws=ws, stream=side)
+                        vd.run_pipeline(plan, col, n, out=out, ws=pws, stream=side)
+            graphs[name] = g
+        stream.wait_stream(side)
         torch.cuda.synchronize()
         r = {}
         for cold in (False, True):
-            for name, f in list(calls.items()) + [("step", lambda: [g() for g in calls.values()])]:
+            for name, g in graphs.items():
+                f = g.replay
                 ev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True))
                       for _ in range(steps)]
                 for i in range(steps):
@@ -771,7 +793,8 @@ def c1_main(args, rank, world, local):
                 torch.cuda.synchronize()
                 us = sorted(a.elapsed_time(b) * 1e3 for a, b in ev)
                 r[f"{name}_{'cold' if cold else 'warm'}_us"] = {"median": statistics.median(us), "best": us[0]}
-        launches += vd.last_launch_count()
+        launches = max(launches, nl)
+        r["launches_per_step"] = nl
         # parity with the oracle (count, positions, f64 sum within 1e-9)
         c = int(cnt.item())
         pos_o, cnt_o, (sh, sl) = oracle.select_f32(v.cpu().numpy(), t, "lt")
@@ -849,8 +872,12 @@ def fig14_main(args, rank, world, local):
     Loop (vd_gather_multi), Separate Loops (one vd_gather per column), or a
     Layout Transform (vd_zip of the target into 8-byte rows, inside the timed
     step, then vd_gather_rows).  Lookups are sequential (i mod m) or uniform
-    random.  Algorithmic bytes per position: 4 (pos) + 2 x 4 gathered + 2 x 4
-    written = 20 B."""
+    random.  Algorithmic bytes (reading A35, the rule Fig 16 uses, A33): per
+    position 4 B read + 2 x 4 B written; a random lookup into a target
+    column larger than L2 moves one 64-byte HBM block per column it touches
+    (Single / Separate: 2 blocks, Layout: 1 block of the zipped row), plus
+    the zip pass's 16 B per target row; sequential lookups and targets that
+    fit L2 read the target once (8 B per target row)."""
     import torch
 
     import gen
@@ -910,18 +937,27 @@ def fig14_main(args, rank, world, local):
     torch.cuda.synchronize()
     clk = clocks.stop()
     ms = comm.max([e0.elapsed_time(e1) / steps])[0]
-    peak, kind = hbm_peak()
-    alg = 20 * n / (ms * 1e-3) / 1e9
+    col_bytes = m * 4
+    big = args.pattern == "random" and col_bytes > 126 * (1 << 20)
+    if big:
+        look = (64 if args.strategy == "layout" else 128) * n
+    else:
+        look = 8 * m
+    zip_b = 16 * m if args.strategy == "layout" else 0
+    alg_bytes = 12 * n + look + zip_b
+    alg = alg_bytes / (ms * 1e-3) / 1e9
     line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
             "vs_baseline": None, "dtype": "int32", "data": "synthetic (uniform int32 target, gen/vd_gen.h)",
             "config": {"workload": f"fig14_{args.strategy}_{args.pattern}_{args.target_mb}MB_{n_total}",
                        "strategy": args.strategy, "pattern": args.pattern, "target_mb": args.target_mb,
-                       "positions": n_total, "l2": "positions + outputs 2.4 GB per step > 126 MB L2"},
-            "roofline": {"bound": "hbm", "achieved": alg, "peak": peak, "unit": "GB/s", "frac": alg / peak,
-                         "peak_kind": kind, "traffic": None, "bytes_per_row": 20,
-                         "kernel": {"single": "k_gather", "separate": "k_gather x2",
-                                    "layout": "k_zip + k_gather_rows"}[args.strategy], "kernel_ms": ms},
+                       "positions": n_total, "target_column_mb": col_bytes / 2**20,
+                       "l2": "positions + outputs 2.4 GB per step > 126 MB L2"},
+            "roofline": hbm_roofline(alg, {"single": "k_gather", "separate": "k_gather x2",
+                                           "layout": "k_zip + k_gather_rows"}[args.strategy], ms, None,
+                                     bytes_per_row=alg_bytes / n, lookup_model=(
+                                         "64 B HBM block per column lookup (A33/A35)" if big else
+                                         "target read once (sequential or L2-resident)")),
             "clocks": clk, "e2e": None, "gpu_launches": launches * steps, "result_ok": ok}
     if rank == 0:
         print(json.dumps(line), flush=True)
@@ -989,44 +1025,79 @@ def q15_main(args, rank, world, local, sf):
     """NEXT-4: TPC-H Q15's revenue view -- shipdate in [1996-01-01,
     1996-04-01), GROUP BY l_suppkey (10,000 x SF groups: a key domain far
     beyond a shared-memory table), SUM(ext * (100 - disc)), COUNT(*) --
-    through vd_group_fold (one streaming pass into the min/max-sized global
-    table + the FoldSelect compaction).  Algorithmic bytes: the four columns,
-    dense, 24 B/row (branching late loads touch fewer sectors)."""
+    through vd_group_fold (identity hashing over min..max, one streaming pass
+    into the global table + the FoldSelect compaction) or, with
+    --grouping hash, vd_hash_group_fold (open addressing, shared-memory tables
+    spilling to a global one, sized from the distinct-key bound).  N > 1: row
+    ranges per rank; every rank's compacted groups go into a fixed-stride
+    buffer, one all-gather (counts + groups), then vd_merge_groups (the
+    cross-GPU merge of compacted groups, 128-bit sums) -- the step ends with
+    the merged groups on every rank.  Algorithmic bytes (A31): the filter
+    column in full and, of the other columns, the 64-byte blocks holding a
+    qualifying row."""
     import torch
 
     import gen
     from paper_journals_pvldb_pirkmzm16_b200 import vd
 
-    if world > 1:
-        if rank == 0:
-            print(json.dumps({"metric": METRIC, "workload": "q15", "unavailable": "q15 runs on one GPU "
-                              "(a cross-GPU merge of compacted high-cardinality groups is not implemented)"}))
-        return
     torch.cuda.set_device(local % torch.cuda.device_count())
     dev = torch.device("cuda", local % torch.cuda.device_count())
+    comm = Comm(world, args.dist_backend, dev)
     stream = torch.cuda.current_stream()
-    n = gen.lineitem_rows(sf)
+    n_total = gen.lineitem_rows(sf)
+    a0, b0 = rank * n_total // world, (rank + 1) * n_total // world
+    n = b0 - a0
     names = ["l_shipdate", "l_suppkey", "l_extendedprice", "l_discount"]
     cols = []
     for nm in names:
         col = gen.LINEITEM_COLS[nm]
         t = torch.empty(n, dtype=getattr(torch, _dt(col)), device=dev)
-        gen.device(col, t.data_ptr(), n, 0, sf=sf, seed=args.seed, stream=stream.cuda_stream)
+        gen.device(col, t.data_ptr(), n, a0, sf=sf, seed=args.seed, stream=stream.cuda_stream)
         cols.append(t)
     torch.cuda.synchronize()
     views = [vd.describe(t, stream=stream) for t in cols]
+    # every rank sizes its table from the key column's global domain (the
+    # supplier table's key range: 1 .. 10000 x SF), so strides agree
+    kmin, kmax = 1, gen.supplier_rows(sf)
+    views[1].min, views[1].max, views[1].has_minmax = kmin, kmax, 1
     p = vd.pred([[(0, ">=", 9496), (0, "<", 9587)]])
     aggs = [("sum", [2, (3, 100, -1)]), ("count",)]
-    D = views[1].max - views[1].min + 1
+    D = kmax - kmin + 1
+    hashed = args.grouping == "hash"
     keys = torch.empty(D, dtype=torch.int64, device=dev)
     rows = torch.empty(D, dtype=torch.int64, device=dev)
     slots = torch.empty(D * len(aggs) * 16, dtype=torch.uint8, device=dev)
-    ng = torch.empty(1, dtype=torch.int64, device=dev)
-    ws = vd.alloc_ws(vd.group_fold_ws_bytes(D, len(aggs)), dev)
+    ng = torch.zeros(1, dtype=torch.int64, device=dev)
+    if hashed:
+        ws = vd.alloc_ws(vd.hash_group_fold_ws_bytes(D, len(aggs)), dev)
+    else:
+        ws = vd.alloc_ws(vd.group_fold_ws_bytes(D, len(aggs)), dev)
+    if world > 1:
+        gk = torch.empty(D * world, dtype=torch.int64, device=dev)
+        gr = torch.empty(D * world, dtype=torch.int64, device=dev)
+        gs = torch.empty(D * world * len(aggs) * 16, dtype=torch.uint8, device=dev)
+        gn = torch.empty(world, dtype=torch.int64, device=dev)
+        mk = torch.empty(D, dtype=torch.int64, device=dev)
+        mr = torch.empty(D, dtype=torch.int64, device=dev)
+        ms_ = torch.empty(D * len(aggs) * 16, dtype=torch.uint8, device=dev)
+        mn = torch.empty(1, dtype=torch.int64, device=dev)
+        mws = vd.alloc_ws(vd.merge_groups_ws_bytes(D, len(aggs)), dev)
 
     def step():
-        vd.group_fold(views, n, 1, aggs, p, out_keys=keys, out_aggs=slots, out_rows=rows, out_ngroups=ng, ws=ws,
-                      stream=stream)
+        if hashed:
+            vd.hash_group_fold(views, n, 1, aggs, p, max_groups=D, out_keys=keys, out_aggs=slots, out_rows=rows,
+                               out_ngroups=ng, ws=ws, stream=stream)
+        else:
+            vd.group_fold(views, n, 1, aggs, p, out_keys=keys, out_aggs=slots, out_rows=rows, out_ngroups=ng,
+                          ws=ws, stream=stream)
+        if world > 1:
+            comm.all_gather(ng, gn)
+            comm.all_gather(keys, gk)
+            comm.all_gather(rows, gr)
+            comm.all_gather(slots, gs)
+            vd.merge_groups(gk, gs, gr, gn, world, D, [vd.VD_AGG_SUM, vd.VD_AGG_COUNT], [False, False],
+                            max_groups=D, out_keys=mk, out_aggs=ms_, out_rows=mr, out_ngroups=mn, ws=mws,
+                            stream=stream)
 
     for _ in range(max(args.warmup, 3)):
         step()
@@ -1036,6 +1107,7 @@ def q15_main(args, rank, world, local, sf):
     clocks = ClockSampler(local)
     clocks.start()
     time.sleep(0.3)
+    comm.barrier()
     torch.cuda.synchronize()
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     e0.record(stream)
@@ -1043,14 +1115,16 @@ def q15_main(args, rank, world, local, sf):
         step()
     e1.record(stream)
     torch.cuda.synchronize()
+    comm.barrier()
     clk = clocks.stop()
-    ms = e0.elapsed_time(e1) / steps
-    g = int(ng.item())
-    digest = __import__("hashlib").sha256(keys[:g].cpu().numpy().tobytes() + rows[:g].cpu().numpy().tobytes() +
-                                          slots[:g * 32].cpu().numpy().tobytes()).hexdigest()[:16]
-    # algorithmic bytes of the branching plan: the filter column in full, and
-    # of every other column the 64-byte DRAM blocks holding a qualifying row
-    # (HBM's access granule; the dense figure, 24 B/row, is the predicated plan's)
+    ms = comm.max([e0.elapsed_time(e1) / steps])[0]
+    rk, rr, rs, rn = (mk, mr, ms_, mn) if world > 1 else (keys, rows, slots, ng)
+    g = int(rn.item())
+    order = torch.argsort(rk[:g])  # a canonical order for the digest (hash output is in table order)
+    kk = rk[:g][order].cpu().numpy()
+    rowsv = rr[:g][order].cpu().numpy()
+    sl = rs[:g * 32].view(g, 32)[order].cpu().numpy()
+    digest = __import__("hashlib").sha256(kk.tobytes() + rowsv.tobytes() + sl.tobytes()).hexdigest()[:16]
     mask = (cols[0] >= 9496) & (cols[0] < 9587)
     alg_bytes = 4 * n
     for t in cols[1:]:
@@ -1059,22 +1133,25 @@ def q15_main(args, rank, world, local, sf):
         alg_bytes += 64 * (int(m.sum().item()) + int(bool(mask[n // r * r:].any().item())))
     sel = float(mask.float().mean().item())
     del mask
-    peak, kind = hbm_peak()
     alg = alg_bytes / (ms * 1e-3) / 1e9
-    line = {"metric": METRIC, "value": n / (ms * 1e-3), "unit": "rows/s", "n_gpus": 1, "steps": steps,
+    line = {"metric": METRIC, "value": n_total / (ms * 1e-3), "unit": "rows/s", "n_gpus": world, "steps": steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
             "vs_baseline": None, "dtype": "int64",
             "data": "synthetic (dbgen-shaped, counter-based generator gen/vd_gen.h, generated in HBM)",
-            "config": bench_config(args, "q15", sf, 1), "groups_domain": D, "groups": g,
-            "roofline": hbm_roofline(alg, "vd_group_fold (k_grp_init + k_grp_fold + compaction)", ms,
-                                     ncu_traffic("q15"), bytes_per_row=alg_bytes / n, dense_bytes_per_row=24,
+            "config": {**bench_config(args, "q15", sf, world), "grouping": args.grouping}, "groups_domain": D,
+            "groups": g,
+            "roofline": hbm_roofline(alg, ("vd_hash_group_fold" if hashed else "vd_group_fold") +
+                                     (" + all-gather + vd_merge_groups" if world > 1 else ""), ms,
+                                     ncu_traffic("q15", world), bytes_per_row=alg_bytes / n, dense_bytes_per_row=24,
                                      selectivity=sel),
             "clocks": clk, "e2e": None, "gpu_launches": launches * steps, "result_digest": digest}
-    if not args.no_cpu_baseline:
+    if rank == 0 and world == 1 and not args.no_cpu_baseline:
         cb = cpu_baseline("q15", sf, args.seed, args.cpu_seconds, args.selectivity, n)
         if cb is not None:
             line["cpu_baseline"] = cb
-    print(json.dumps(line), flush=True)
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    comm.close()
 
 
 def _dt(col):
@@ -1149,7 +1226,7 @@ def bench_config(args, w, sf, world):
             "selagg": f"selagg_f32x2_{n_total}_s{args.selectivity:g}",
             "selpos": f"selpos_f32_{n_total}_s{args.selectivity:g}",
             "c1": f"c1_select_f32_{n_total}_s{args.selectivity:g}",
-            "fkjsel": f"fkjsel_{n_total}x16777216_s{args.selectivity:g}"}.get(w, w)
+            "fkjsel": f"fkjsel_{n_total}x{128 * 1024 * 1024}_s{args.selectivity:g}"}.get(w, w)
     per_gpu = n_total // world
     return {"workload": name, "rows": n_total, "rows_per_gpu": per_gpu, "sf": sf, "sel_mode": args.sel_mode,
             **({"materialize": args.materialize, "chunk": args.chunk} if args.materialize != "none" else {}),

@@ -472,22 +472,25 @@ vd_status vd_hash_group_fold(const vd_column* cols, int32_t ncols, int64_t n, co
                              int64_t* out_rows, int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
 
 /* Cross-GPU merge of COMPACTED groups (the Fig 3 hierarchical fold one
- * level above GPUs, for high-cardinality grouping): `ngroups`
- * (host count) groups -- e.g. every rank's vd_group_fold / vd_hash_group_fold
- * output, concatenated after an all-gather -- are re-inserted into one hash
- * table: equal keys combine (integer SUM / COUNT exactly in 128 bits, float
- * SUM in f64 in an unspecified order, MIN / MAX over the non-epsilon
- * values, row counts added) and the result is compacted in table order.
- *   keys / aggs / rows : device, the vd_group_fold output layout (16-byte
- *       aggregate slots, naggs per group).
+ * level above GPUs, for high-cardinality grouping): nparts
+ * blocks of `stride` groups each -- e.g. every rank's vd_group_fold /
+ * vd_hash_group_fold output after an all-gather of fixed-size buffers,
+ * block r holding counts_dev[r] valid groups and padding after them -- are
+ * re-inserted into one hash table: equal keys combine (integer SUM / COUNT
+ * exactly in 128 bits, float SUM in f64 in an unspecified order, MIN / MAX
+ * over the non-epsilon values, row counts added) and the result is
+ * compacted in table order.
+ *   keys / aggs / rows : device, [nparts * stride] groups in the
+ *       vd_group_fold output layout (16-byte aggregate slots, naggs each).
+ *   counts_dev : device int64 [nparts], valid groups per block (<= stride).
  *   kinds_host[a] / isf_host[a] : aggregate kind and whether it is f64.
  *   max_groups : bound on the distinct keys; *out_ngroups_dev = -1 if exceeded.
  *   ws : vd_merge_groups_ws_bytes(max_groups, naggs). */
 vd_status vd_merge_groups_ws_bytes(int64_t max_groups, int32_t naggs, size_t* bytes_host);
-vd_status vd_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, int64_t ngroups,
-                          const int32_t* kinds_host, const int32_t* isf_host, int32_t naggs, int64_t max_groups,
-                          int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ngroups_dev, void* ws,
-                          size_t ws_bytes, void* stream);
+vd_status vd_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, const int64_t* counts_dev,
+                          int32_t nparts, int64_t stride, const int32_t* kinds_host, const int32_t* isf_host,
+                          int32_t naggs, int64_t max_groups, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
+                          int64_t* out_ngroups_dev, void* ws, size_t ws_bytes, void* stream);
 
 /* Compacted result of a pipeline: the FoldSelect compaction of Fig 11
  * applied to the merged partials -- the non-empty groups

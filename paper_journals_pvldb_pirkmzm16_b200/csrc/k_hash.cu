@@ -335,9 +335,11 @@ __global__ void __launch_bounds__(HG_THREADS) k_hg_emit(const int64_t* __restric
 // ---- cross-GPU merge of compacted groups ------------------------------------------
 struct HmArgs {
     const int64_t* in_keys;
-    const unsigned long long* in_aggs;  // [m][naggs] 16-byte slots
+    const unsigned long long* in_aggs;  // [nparts * stride][naggs] 16-byte slots
     const int64_t* in_rows;
-    int64_t m;
+    const int64_t* in_counts;           // [nparts] valid groups per part
+    int64_t stride;                     // groups per part block
+    int64_t m;                          // nparts * stride
     int32_t naggs;
     int32_t kind[VD_MAX_AGGS], isf[VD_MAX_AGGS];
     uint64_t mask;
@@ -368,6 +370,8 @@ __global__ void __launch_bounds__(HG_THREADS) k_hm_insert(const __grid_constant_
     g.keys = a.keys;
     g.overflow = a.overflow;
     for (int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x; i < a.m; i += (int64_t)gridDim.x * blockDim.x) {
+        const int64_t part = i / a.stride;
+        if (i - part * a.stride >= __ldg(a.in_counts + part)) continue;  // padding past the part's groups
         const int64_t key = a.in_keys[i];
         const int64_t s = hg_global_slot(g, key);
         if (s < 0) continue;
@@ -495,15 +499,18 @@ cudaError_t launch_hash_group_fold(const DevCols& cols, const DevPred& pred, int
     return hg_compact(L, e, out_keys, out_aggs, out_rows, out_ng, s, nl);
 }
 
-cudaError_t launch_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, int64_t m,
-                                const int32_t* kinds, const int32_t* isf, int naggs, int64_t est, int64_t* out_keys,
-                                void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws, cudaStream_t s,
-                                int* nl) {
+cudaError_t launch_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, const int64_t* counts,
+                                int nparts, int64_t stride, const int32_t* kinds, const int32_t* isf, int naggs,
+                                int64_t est, int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ng,
+                                void* ws, cudaStream_t s, int* nl) {
     HmArgs A;
     std::memset(&A, 0, sizeof(A));
     A.in_keys = keys;
     A.in_aggs = (const unsigned long long*)aggs;
     A.in_rows = rows;
+    A.in_counts = counts;
+    A.stride = stride;
+    const int64_t m = (int64_t)nparts * stride;
     A.m = m;
     A.naggs = naggs;
     HgEmit e;

@@ -804,16 +804,17 @@ vd_status vd_merge_groups_ws_bytes(int64_t max_groups, int32_t naggs, size_t* by
     return VD_OK;
 }
 
-vd_status vd_merge_groups(const int64_t* keys, const void* aggs_in, const int64_t* rows, int64_t ngroups,
-                          const int32_t* kinds_host, const int32_t* isf_host, int32_t naggs, int64_t max_groups,
-                          int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ngroups, void* ws,
-                          size_t ws_bytes, void* stream) {
+vd_status vd_merge_groups(const int64_t* keys, const void* aggs_in, const int64_t* rows, const int64_t* counts_dev,
+                          int32_t nparts, int64_t stride, const int32_t* kinds_host, const int32_t* isf_host,
+                          int32_t naggs, int64_t max_groups, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
+                          int64_t* out_ngroups, void* ws, size_t ws_bytes, void* stream) {
     reset_launches();
-    if (ngroups < 0) return VD_E_SHAPE;
+    if (nparts < 0 || stride < 0) return VD_E_SHAPE;
     if (naggs < 0 || naggs > VD_MAX_AGGS || (naggs > 0 && (!kinds_host || !isf_host))) return VD_E_ARG;
     if (max_groups < 1 || max_groups > VD_MAX_HASH_GROUPS) { set_error("merge_groups: max_groups"); return VD_E_ARG; }
-    if ((ngroups > 0 && (!keys || !rows || (naggs > 0 && !aggs_in))) || !out_keys || !out_rows || !out_ngroups ||
-        (naggs > 0 && !out_aggs))
+    const bool any = nparts > 0 && stride > 0;
+    if ((any && (!keys || !rows || !counts_dev || (naggs > 0 && !aggs_in))) || !out_keys || !out_rows ||
+        !out_ngroups || (naggs > 0 && !out_aggs))
         return VD_E_NULL;
     for (int a = 0; a < naggs; ++a) {
         if (kinds_host[a] < VD_AGG_SUM || kinds_host[a] > VD_AGG_MAX) { set_error("bad aggregate kind"); return VD_E_ARG; }
@@ -826,8 +827,9 @@ vd_status vd_merge_groups(const int64_t* keys, const void* aggs_in, const int64_
     if ((st = check_ws(ws, ws_bytes, hash_group_ws_bytes(max_groups, naggs, true))) != VD_OK) return st;
     if ((st = check_device()) != VD_OK) return st;
     int nl = 0;
-    st = cuda_status(launch_merge_groups(keys, aggs_in, rows, ngroups, kinds_host, isf_host, naggs, max_groups,
-                                         out_keys, out_aggs, out_rows, out_ngroups, ws, (cudaStream_t)stream, &nl));
+    st = cuda_status(launch_merge_groups(keys, aggs_in, rows, counts_dev, any ? nparts : 0, any ? stride : 0,
+                                         kinds_host, isf_host, naggs, max_groups, out_keys, out_aggs, out_rows,
+                                         out_ngroups, ws, (cudaStream_t)stream, &nl));
     count_launches(nl);
     return st;
 }

@@ -117,10 +117,10 @@ cudaError_t launch_hash_group_fold(const DevCols& cols, const DevPred& pred, int
                                    const vd_agg* aggs, const int32_t* isf, int naggs, int64_t max_groups,
                                    int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws,
                                    cudaStream_t s, int* nl);
-cudaError_t launch_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, int64_t m,
-                                const int32_t* kinds, const int32_t* isf, int naggs, int64_t max_groups,
-                                int64_t* out_keys, void* out_aggs, int64_t* out_rows, int64_t* out_ng, void* ws,
-                                cudaStream_t s, int* nl);
+cudaError_t launch_merge_groups(const int64_t* keys, const void* aggs, const int64_t* rows, const int64_t* counts,
+                                int nparts, int64_t stride, const int32_t* kinds, const int32_t* isf, int naggs,
+                                int64_t max_groups, int64_t* out_keys, void* out_aggs, int64_t* out_rows,
+                                int64_t* out_ng, void* ws, cudaStream_t s, int* nl);
 
 int num_sms();
 

@@ -92,8 +92,9 @@ def q9(sel_mode=VD_SEL_BRANCH, force_generic=False):
                     aggs=[("sum", [2, (3, 100, -1)]), ("count",)], force_generic=force_generic)
 
 
-# Fig 16 selective FK join: a 128 MB target (16 M int64 rows), larger than the 126 MB L2
-FKJSEL_TARGET_ROWS = 16 * 1024 * 1024
+# Fig 16 selective FK join: a 1 GiB target (128 Mi int64 rows), far larger than the 126 MB L2
+# (a 128 MB target is about L2-sized: its lookups hit L2 and overstate the HBM fraction)
+FKJSEL_TARGET_ROWS = 128 * 1024 * 1024
 FKJSEL_VMAX = 1_000_000
 
 

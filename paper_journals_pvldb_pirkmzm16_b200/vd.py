@@ -143,8 +143,9 @@ _sigs = {
     "vd_hash_group_fold": (c_int32, [_P(vd_column), c_int32, c_int64, _P(vd_pred), c_int32, _P(vd_agg), c_int32,
                                      c_int64, c_void_p, c_void_p, c_void_p, c_void_p, c_void_p, c_size_t, c_void_p]),
     "vd_merge_groups_ws_bytes": (c_int32, [c_int64, c_int32, _P(c_size_t)]),
-    "vd_merge_groups": (c_int32, [c_void_p, c_void_p, c_void_p, c_int64, _P(c_int32), _P(c_int32), c_int32, c_int64,
-                                  c_void_p, c_void_p, c_void_p, c_void_p, c_void_p, c_size_t, c_void_p]),
+    "vd_merge_groups": (c_int32, [c_void_p, c_void_p, c_void_p, c_void_p, c_int32, c_int64, _P(c_int32), _P(c_int32),
+                                  c_int32, c_int64, c_void_p, c_void_p, c_void_p, c_void_p, c_void_p, c_size_t,
+                                  c_void_p]),
     "vd_last_launch_count": (c_int32, []),
     "vd_last_fragment": (ctypes.c_char_p, []),
     "vd_abi_struct_sizes": (c_int32, [_P(c_size_t), c_int32]),
@@ -551,15 +552,25 @@ def group_fold(cols: Sequence[vd_column], n: int, key_col: int, aggs=(), pred_: 
                          ws.data_ptr(), ws.numel(), _stream(stream)), "vd_group_fold")
 
 
+def hash_group_fold_ws_bytes(max_groups: int, naggs: int) -> int:
+    b = c_size_t(0)
+    _ok(_L.vd_hash_group_fold_ws_bytes(max_groups, naggs, ctypes.byref(b)), "vd_hash_group_fold_ws_bytes")
+    return int(b.value)
+
+
+def merge_groups_ws_bytes(max_groups: int, naggs: int) -> int:
+    b = c_size_t(0)
+    _ok(_L.vd_merge_groups_ws_bytes(max_groups, naggs, ctypes.byref(b)), "vd_merge_groups_ws_bytes")
+    return int(b.value)
+
+
 def hash_group_fold(cols: Sequence[vd_column], n: int, key_col: int, aggs=(), pred_: Optional[vd_pred] = None, *,
                     max_groups: int, out_keys, out_aggs, out_rows, out_ngroups, ws=None, stream=None):
     """vd_hash_group_fold (NEXT-4, sparse keys): open-addressing table sized
     from max_groups (an upper bound on the distinct keys); groups come out in
     table order; out_ngroups[0] = -1 if the table filled up."""
     if ws is None:
-        b = c_size_t(0)
-        _ok(_L.vd_hash_group_fold_ws_bytes(max_groups, len(aggs), ctypes.byref(b)), "vd_hash_group_fold_ws_bytes")
-        ws = alloc_ws(int(b.value), out_keys.device)
+        ws = alloc_ws(hash_group_fold_ws_bytes(max_groups, len(aggs)), out_keys.device)
     arr = _cols_array(cols)
     ag = aggs_array(aggs)
     _ok(_L.vd_hash_group_fold(arr, len(cols), n, ctypes.byref(pred_) if pred_ is not None else None, key_col, ag,
@@ -568,20 +579,21 @@ def hash_group_fold(cols: Sequence[vd_column], n: int, key_col: int, aggs=(), pr
         "vd_hash_group_fold")
 
 
-def merge_groups(keys, aggs_slots, rows, ngroups: int, kinds: Sequence[int], float_aggs: Sequence[bool], *,
-                 max_groups: int, out_keys, out_aggs, out_rows, out_ngroups, ws=None, stream=None):
-    """vd_merge_groups: the cross-GPU merge of compacted groups (device tensors
-    in the vd_group_fold layout, e.g. every rank's output concatenated)."""
+def merge_groups(keys, aggs_slots, rows, counts, nparts: int, stride: int, kinds: Sequence[int],
+                 float_aggs: Sequence[bool], *, max_groups: int, out_keys, out_aggs, out_rows, out_ngroups, ws=None,
+                 stream=None):
+    """vd_merge_groups: the cross-GPU merge of compacted groups -- nparts
+    blocks of `stride` groups (device tensors in the vd_group_fold layout,
+    e.g. an all-gather of every rank's padded output), block r holding
+    counts[r] (device int64 tensor) valid groups."""
     na = len(kinds)
     if ws is None:
-        b = c_size_t(0)
-        _ok(_L.vd_merge_groups_ws_bytes(max_groups, na, ctypes.byref(b)), "vd_merge_groups_ws_bytes")
-        ws = alloc_ws(int(b.value), out_keys.device)
+        ws = alloc_ws(merge_groups_ws_bytes(max_groups, na), out_keys.device)
     k = (c_int32 * max(1, na))(*kinds)
     f = (c_int32 * max(1, na))(*[int(bool(x)) for x in float_aggs] + [0] * (na - len(float_aggs)))
-    _ok(_L.vd_merge_groups(_ptr(keys), _ptr(aggs_slots), _ptr(rows), ngroups, k, f, na, max_groups,
-                           out_keys.data_ptr(), _ptr(out_aggs), out_rows.data_ptr(), out_ngroups.data_ptr(),
-                           ws.data_ptr(), ws.numel(), _stream(stream)), "vd_merge_groups")
+    _ok(_L.vd_merge_groups(_ptr(keys), _ptr(aggs_slots), _ptr(rows), _ptr(counts), nparts, stride, k, f, na,
+                           max_groups, out_keys.data_ptr(), _ptr(out_aggs), out_rows.data_ptr(),
+                           out_ngroups.data_ptr(), ws.data_ptr(), ws.numel(), _stream(stream)), "vd_merge_groups")
 
 
 def decode_group_slots(buf: bytes, ngroups: int, naggs: int, float_aggs: Sequence[bool] = ()):

@@ -49,7 +49,7 @@ def table(files):
 def fig14():
     """Fig 14: strategy x lookup pattern x target size."""
     for pattern in ["sequential", "random"]:
-        for mb in [4, 128]:
+        for mb in [4, 1024]:
             for strat in ["single", "separate", "layout"]:
                 cmd = [sys.executable, os.path.join(ROOT, "bench.py"), "--workload", "fig14", "--strategy", strat,
                        "--pattern", pattern, "--target-mb", str(mb), "--steps", "30"]

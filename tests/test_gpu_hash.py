@@ -156,23 +156,26 @@ def test_merge_groups_of_shards_equals_whole(G):
     views = [vd.describe(t) for t in keep]
     p = vd.pred([[(0, ">=", Q15_D0), (0, "<", Q15_D1)]])
     aggs = [("sum", [2, (3, 100, -1)]), ("count",)]
-    ks, ss, rs = [], [], []
+    # every "rank" writes into its block of fixed stride (an all-gather of
+    # fixed-size buffers leaves them so), its group count into counts[r]
+    stride = 20000
+    allk = torch.zeros(G * stride, dtype=torch.int64, device="cuda")
+    allr = torch.zeros(G * stride, dtype=torch.int64, device="cuda")
+    alls = torch.zeros(G * stride * 2 * 16, dtype=torch.uint8, device="cuda")
+    counts = torch.zeros(G, dtype=torch.int64, device="cuda")
     for r in range(G):
         a, b = r * n // G, (r + 1) * n // G
         sv = [vd.column(t[a:b], minmax=(v.min, v.max), noeps=bool(v.flags & vd.VD_COL_NOEPS))
               for t, v in zip(keep, views)]
-        dkeys, dslots, drows, g, *_ = run_hash(sv, b - a, 1, aggs, p, max_groups=20000)
-        ks.append(dkeys)
-        ss.append(dslots)
-        rs.append(drows)
-    allk, alls, allr = torch.cat(ks), torch.cat(ss), torch.cat(rs)
-    m = allk.numel()
-    ok = torch.empty(m, dtype=torch.int64, device="cuda")
-    orows = torch.empty(m, dtype=torch.int64, device="cuda")
-    oslots = torch.empty(max(1, m * 2 * 16), dtype=torch.uint8, device="cuda")
+        vd.hash_group_fold(sv, b - a, 1, aggs, p, max_groups=stride, out_keys=allk[r * stride:(r + 1) * stride],
+                           out_aggs=alls[r * stride * 32:(r + 1) * stride * 32],
+                           out_rows=allr[r * stride:(r + 1) * stride], out_ngroups=counts[r:r + 1])
+    ok = torch.empty(stride, dtype=torch.int64, device="cuda")
+    orows = torch.empty(stride, dtype=torch.int64, device="cuda")
+    oslots = torch.empty(stride * 2 * 16, dtype=torch.uint8, device="cuda")
     ong = torch.empty(1, dtype=torch.int64, device="cuda")
-    vd.merge_groups(allk, alls, allr, m, [vd.VD_AGG_SUM, vd.VD_AGG_COUNT], [False, False], max_groups=20000,
-                    out_keys=ok, out_aggs=oslots, out_rows=orows, out_ngroups=ong)
+    vd.merge_groups(allk, alls, allr, counts, G, stride, [vd.VD_AGG_SUM, vd.VD_AGG_COUNT], [False, False],
+                    max_groups=stride, out_keys=ok, out_aggs=oslots, out_rows=orows, out_ngroups=ong)
     torch.cuda.synchronize()
     g = int(ong.item())
     vals = vd.decode_group_slots(oslots[:g * 32].cpu().numpy().tobytes(), g, 2)
