@@ -33,7 +33,7 @@ __device__ __forceinline__ void gather_one(const T* __restrict__ src, int64_t le
 #pragma unroll
     for (int u = 0; u < GATHER_ILP; ++u) {
         bool ok = i[u] < n && p[u] >= 0 && p[u] < len;
-        v[u] = ok ? __ldg(src + p[u]) : Eps<T>::value();
+        v[u] = ok ? ldg64b(src + p[u]) : Eps<T>::value();
     }
 #pragma unroll
     for (int u = 0; u < GATHER_ILP; ++u)
@@ -86,7 +86,7 @@ __global__ void __launch_bounds__(GATHER_THREADS) k_gather_u(GatherArgs g, const
 #pragma unroll
             for (int u = 0; u < GU_ILP; ++u) {
                 const bool ok = p[u] >= 0 && p[u] < g.len[k];
-                v[k][u] = ok ? __ldg((const T*)g.src[k] + p[u]) : Eps<T>::value();
+                v[k][u] = ok ? ldg64b((const T*)g.src[k] + p[u]) : Eps<T>::value();
             }
         __syncwarp();  // all loads issued before the first store
 #pragma unroll
@@ -205,7 +205,7 @@ __global__ void __launch_bounds__(256) k_zip(const __grid_constant__ RowArgs a, 
 template <int NW>
 __device__ __forceinline__ void load_row(const uint64_t* rows, int64_t p, bool ok, uint64_t (&w)[NW]) {
     if (NW == 1) {
-        w[0] = ok ? __ldg(rows + p) : 0;
+        w[0] = ok ? ldg64b(rows + p) : 0;
     } else {
 #pragma unroll
         for (int k = 0; k < NW; k += 2) {

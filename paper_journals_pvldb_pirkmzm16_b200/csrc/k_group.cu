@@ -64,7 +64,9 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_init(const __grid_constant_
     }
 }
 
-// value of aggregate ag at row: product of factors; eps if a factor is epsilon
+// value of aggregate ag at row: product of factors; eps if a factor is epsilon.
+// The row is a qualifying row, loaded late: one 64-byte block per factor
+// column (fetch_typed_64b), not the default 128-byte line.
 __device__ __forceinline__ bool grp_value(const GrpArgs& a, int ag, int64_t row, int64_t* vi, double* vf) {
     bool eps = false;
     if (a.isf[ag]) {
@@ -72,7 +74,7 @@ __device__ __forceinline__ bool grp_value(const GrpArgs& a, int ag, int64_t row,
         for (int f = 0; f < a.nf[ag]; ++f) {
             double x = 0;
             if (a.fcol[ag][f] >= 0) {
-                const Val c = fetch_typed(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
+                const Val c = fetch_typed_64b(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
                 eps |= c.eps;
                 x = c.isf ? c.f : (double)c.i;
             }
@@ -84,7 +86,7 @@ __device__ __forceinline__ bool grp_value(const GrpArgs& a, int ag, int64_t row,
         for (int f = 0; f < a.nf[ag]; ++f) {
             int64_t x = 0;
             if (a.fcol[ag][f] >= 0) {
-                const Val c = fetch_typed(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
+                const Val c = fetch_typed_64b(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
                 eps |= c.eps;
                 x = c.i;
             }
@@ -95,7 +97,24 @@ __device__ __forceinline__ bool grp_value(const GrpArgs& a, int ag, int64_t row,
     return !eps;
 }
 
+// one table update: a global reduction that keeps the table's line in L2
+// (evict_last) while the scan streams past it (evict_first)
+__device__ __forceinline__ void grp_red(unsigned long long* slot, int kind, int isf, int64_t vi, double vf,
+                                        uint64_t pol) {
+    if (kind == VD_AGG_SUM) {
+        if (isf) red_add_f64_hint((double*)slot, vf, pol);
+        else red_add_u64_hint(slot, (unsigned long long)vi, pol);
+    } else if (kind == VD_AGG_MIN) {
+        red_min_s64_hint((long long*)slot, (long long)vi, pol);
+    } else if (kind == VD_AGG_MAX) {
+        red_max_s64_hint((long long*)slot, (long long)vi, pol);
+    } else {
+        red_add_u64_hint(slot, (unsigned long long)vi, pol);  // COUNT / row count
+    }
+}
+
 __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold(const __grid_constant__ GrpArgs a) {
+    const uint64_t pol_t = policy_evict_last();
     const int lane = threadIdx.x & 31;
     const int W = a.naggs + 1;
     const int64_t warps = (int64_t)gridDim.x * (GRP_THREADS / 32);
@@ -105,7 +124,7 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold(const __grid_constant_
         bool ok = row < a.n && eval_pred_row(a.pred, a.cols, row);  // branching: later columns only for qualifying rows
         int64_t g = -1;
         if (ok) {
-            const Val k = fetch_typed(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
+            const Val k = fetch_typed_64b(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
             if (k.eps) ok = false;  // epsilon key: no group (reading A9)
             else g = k.i - a.kmin;  // in [0, D) by the key's metadata
         }
@@ -123,20 +142,11 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold(const __grid_constant_
             const int kind = a.kind[ag];
             if (kind != VD_AGG_COUNT) has = grp_value(a, ag, row, &vi, &vf);
             if (kind == VD_AGG_COUNT) {
-                if (lane == leader) atomicAdd(&slot[ag], (unsigned long long)nm);
+                if (lane == leader) grp_red(&slot[ag], VD_AGG_COUNT, 0, nm, 0, pol_t);
                 continue;
             }
             if (nm == 1) {  // the common case for uniform keys: no shuffles
-                if (has) {
-                    if (kind == VD_AGG_SUM) {
-                        if (a.isf[ag]) atomicAdd((double*)&slot[ag], vf);
-                        else atomicAdd(&slot[ag], (unsigned long long)vi);
-                    } else if (kind == VD_AGG_MIN) {
-                        atomicMin((long long*)&slot[ag], (long long)vi);
-                    } else {
-                        atomicMax((long long*)&slot[ag], (long long)vi);
-                    }
-                }
+                if (has) grp_red(&slot[ag], kind, a.isf[ag], vi, vf, pol_t);
                 continue;
             }
             // combine the group's lanes in lane order (fixed order per warp step)
@@ -154,18 +164,9 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold(const __grid_constant_
                 else if (kind == VD_AGG_MIN) ci = xi < ci ? xi : ci;
                 else ci = xi > ci ? xi : ci;
             }
-            if (lane == leader && any) {
-                if (kind == VD_AGG_SUM) {
-                    if (a.isf[ag]) atomicAdd((double*)&slot[ag], cf);
-                    else atomicAdd(&slot[ag], (unsigned long long)ci);
-                } else if (kind == VD_AGG_MIN) {
-                    atomicMin((long long*)&slot[ag], (long long)ci);
-                } else {
-                    atomicMax((long long*)&slot[ag], (long long)ci);
-                }
-            }
+            if (lane == leader && any) grp_red(&slot[ag], kind, a.isf[ag], ci, cf, pol_t);
         }
-        if (lane == leader) atomicAdd(&slot[a.naggs], (unsigned long long)nm);  // the group's row count
+        if (lane == leader) grp_red(&slot[a.naggs], VD_AGG_COUNT, 0, nm, 0, pol_t);  // the group's row count
     }
 }
 
@@ -185,26 +186,19 @@ struct GrpIv {
     int64_t lo0, hi0, lo1, hi1;
 };
 
-__device__ __forceinline__ void grp_fold_row(const GrpArgs& a, int64_t row) {
-    const Val k = fetch_typed(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
+__device__ __forceinline__ void grp_fold_row(const GrpArgs& a, int64_t row, uint64_t pol_t) {
+    const Val k = fetch_typed_64b(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
     if (k.eps) return;
     unsigned long long* slot = a.table + (size_t)(k.i - a.kmin) * (a.naggs + 1);
     for (int ag = 0; ag < a.naggs; ++ag) {
         const int kind = a.kind[ag];
-        if (kind == VD_AGG_COUNT) { atomicAdd(&slot[ag], 1ull); continue; }
+        if (kind == VD_AGG_COUNT) { grp_red(&slot[ag], VD_AGG_COUNT, 0, 1, 0, pol_t); continue; }
         int64_t vi = 0;
         double vf = 0;
         if (!grp_value(a, ag, row, &vi, &vf)) continue;
-        if (kind == VD_AGG_SUM) {
-            if (a.isf[ag]) atomicAdd((double*)&slot[ag], vf);
-            else atomicAdd(&slot[ag], (unsigned long long)vi);
-        } else if (kind == VD_AGG_MIN) {
-            atomicMin((long long*)&slot[ag], (long long)vi);
-        } else {
-            atomicMax((long long*)&slot[ag], (long long)vi);
-        }
+        grp_red(&slot[ag], kind, a.isf[ag], vi, vf, pol_t);
     }
-    atomicAdd(&slot[a.naggs], 1ull);
+    grp_red(&slot[a.naggs], VD_AGG_COUNT, 0, 1, 0, pol_t);
 }
 
 // Qualifying rows are compacted per warp into a shared-memory stack (ballot
@@ -218,6 +212,7 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold_iv(const __grid_consta
                                                             const __grid_constant__ GrpIv iv) {
     __shared__ int64_t s_q[GRP_THREADS / 32][GRP_QCAP];
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const uint64_t pol_t = policy_evict_last(), pol_s = policy_evict_first();
     int64_t* q_ = s_q[warp];
     int cnt = 0;  // warp-uniform stack depth
     const unsigned lt = lanemask_lt();
@@ -227,10 +222,10 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold_iv(const __grid_consta
             const int64_t row = q_[cnt - k + lane];
             bool ok = true;
             if (iv.c1) {
-                const Val y = fetch_typed(iv.c1, iv.dt1, row);
+                const Val y = fetch_typed_64b(iv.c1, iv.dt1, row);
                 ok = !(y.eps || y.i < iv.lo1 || y.i > iv.hi1);
             }
-            if (ok) grp_fold_row(a, row);
+            if (ok) grp_fold_row(a, row, pol_t);
         }
         cnt -= k;
         __syncwarp();
@@ -242,11 +237,11 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold_iv(const __grid_consta
         int64_t x[4] = {INT64_MIN, INT64_MIN, INT64_MIN, INT64_MIN};
         if (q < nq) {
             if (sizeof(T0) == 4) {
-                const int4 v = ld_stream16((const int32_t*)iv.c0 + 4 * q);
+                const int4 v = ld_stream16_hint((const int32_t*)iv.c0 + 4 * q, pol_s);
                 x[0] = v.x; x[1] = v.y; x[2] = v.z; x[3] = v.w;
             } else {
-                const int4 v0 = ld_stream16((const int64_t*)iv.c0 + 4 * q);
-                const int4 v1 = ld_stream16((const int64_t*)iv.c0 + 4 * q + 2);
+                const int4 v0 = ld_stream16_hint((const int64_t*)iv.c0 + 4 * q, pol_s);
+                const int4 v1 = ld_stream16_hint((const int64_t*)iv.c0 + 4 * q + 2, pol_s);
                 x[0] = (int64_t)((uint64_t)(uint32_t)v0.y << 32 | (uint32_t)v0.x);
                 x[1] = (int64_t)((uint64_t)(uint32_t)v0.w << 32 | (uint32_t)v0.z);
                 x[2] = (int64_t)((uint64_t)(uint32_t)v1.y << 32 | (uint32_t)v1.x);
@@ -272,7 +267,7 @@ __global__ void __launch_bounds__(GRP_THREADS) k_grp_fold_iv(const __grid_consta
                 const Val y = fetch_typed(iv.c1, iv.dt1, row);
                 if (y.eps || y.i < iv.lo1 || y.i > iv.hi1) continue;
             }
-            grp_fold_row(a, row);
+            grp_fold_row(a, row, pol_t);
         }
     }
 }

@@ -95,7 +95,7 @@ __device__ __forceinline__ bool hg_value(const HgArgs& a, int ag, int64_t row, u
         for (int f = 0; f < a.nf[ag]; ++f) {
             double x = 0;
             if (a.fcol[ag][f] >= 0) {
-                const Val c = fetch_typed(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
+                const Val c = fetch_typed_64b(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
                 eps |= c.eps;
                 x = c.isf ? c.f : (double)c.i;
             }
@@ -107,7 +107,7 @@ __device__ __forceinline__ bool hg_value(const HgArgs& a, int ag, int64_t row, u
         for (int f = 0; f < a.nf[ag]; ++f) {
             int64_t x = 0;
             if (a.fcol[ag][f] >= 0) {
-                const Val c = fetch_typed(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
+                const Val c = fetch_typed_64b(a.cols.p[a.fcol[ag][f]], a.cols.dt[a.fcol[ag][f]], row);
                 eps |= c.eps;
                 x = c.i;
             }
@@ -172,7 +172,7 @@ __global__ void __launch_bounds__(HG_THREADS) k_hg_fold(const __grid_constant__ 
         bool ok = row < a.n && eval_pred_row(a.pred, a.cols, row);
         int64_t key = HG_EMPTY;
         if (ok) {
-            const Val k = fetch_typed(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
+            const Val k = fetch_typed_64b(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
             if (k.eps) ok = false;  // epsilon key: no group (A9)
             else key = k.i;
         }

@@ -1466,12 +1466,6 @@ struct LateLead {
 constexpr int LT_MAXTAB = 4;
 constexpr int LT_COMMON = 4;  // = VD_MAX_CONJ
 
-// L2 eviction policy for data re-read by other rows (the dimension lookups).
-__device__ __forceinline__ uint64_t policy_evict_last() {
-    uint64_t p;
-    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
-    return p;
-}
 
 constexpr int LT_THREADS = 256;
 constexpr int LT_QCAP = 32 + 16 * 32;  // < 32 left over + one 16-row step of every lane
@@ -1479,7 +1473,9 @@ constexpr int LT_QCAP = 32 + 16 * 32;  // < 32 left over + one 16-row step of ev
 constexpr int LT_SMEM_MAX = (GF_MAXCOLS + VD_MAX_GATHERS + VD_MAX_AGGS + 1) * LT_THREADS * 8 + (LT_THREADS / 32) * LT_QCAP * 4;
 
 // Late loads of one row go straight to shared memory (cp.async, no
-// registers held while in flight): every referenced base column at once,
+// registers held while in flight; .L2::64B: each moves one 64-byte block,
+// not the default 128-byte line, scripts/ubench_dram_gran.cu): every
+// referenced base column at once,
 // then the lookups they address.  The thread's values live in its column of
 // sv[ref][LT_THREADS] (dynamic reference indices stay in shared memory, not
 // in spilled local memory), widened to int64 with epsilon = INT64_MIN.  A u8
@@ -1488,15 +1484,15 @@ constexpr int LT_SMEM_MAX = (GF_MAXCOLS + VD_MAX_GATHERS + VD_MAX_AGGS + 1) * LT
 __device__ __forceinline__ void lt_cp(int64_t* sdst, const void* col, int32_t dt, int64_t i, int64_t len,
                                       uint64_t pol) {
     if (dt == VD_I64) {
-        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 8, %2;" ::"r"(smem_u32(sdst)),
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint.L2::64B [%0], [%1], 8, %2;" ::"r"(smem_u32(sdst)),
                      "l"((const int64_t*)col + i), "l"(pol)
                      : "memory");
     } else if (dt == VD_I32) {
-        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint.L2::64B [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
                      "l"((const int32_t*)col + i), "l"(pol)
                      : "memory");
     } else if ((i | 3) < len) {
-        asm volatile("cp.async.ca.shared.global.L2::cache_hint [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
+        asm volatile("cp.async.ca.shared.global.L2::cache_hint.L2::64B [%0], [%1], 4, %2;" ::"r"(smem_u32(sdst)),
                      "l"((const uint8_t*)col + (i & ~(int64_t)3)), "l"(pol)
                      : "memory");
     } else {

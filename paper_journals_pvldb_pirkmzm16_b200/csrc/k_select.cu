@@ -531,6 +531,7 @@ constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
 constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
 constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
+constexpr int SC_MAXCH = 12288;              // chunks per CTA (counts kept in shared memory)
 
 template <int MODE>
 __device__ __forceinline__ int sc_stage_positions(const uint32_t (&bw)[32], int64_t row0, int a, int32_t* sw,
@@ -590,13 +591,16 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     extern __shared__ __align__(128) uint8_t smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)SC_STAGES * TB);
     uint64_t* empty = full + SC_STAGES;
+    uint16_t* s_ccnt = reinterpret_cast<uint16_t*>(empty + SC_STAGES);  // per-chunk counts (phase 1 -> 2)
     __shared__ int s_cnt[SC_CW];
+    __shared__ int s_scan[SC_THREADS / 32];
     __shared__ int64_t s_base;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     // the CTA's chunk range [c0, c1) (chunk = 1024 rows), tiles of SC_CHUNKS
     const int64_t nchunks = (n + 1023) / 1024;
     const int64_t c0 = nchunks * blockIdx.x / gridDim.x, c1 = nchunks * (blockIdx.x + 1) / gridDim.x;
-    const int64_t ntile = (c1 - c0 + SC_CHUNKS - 1) / SC_CHUNKS;
+    const int nch = (int)(c1 - c0);  // <= SC_MAXCH (host-checked)
+    const int64_t ntile = (nch + SC_CHUNKS - 1) / SC_CHUNKS;
     if (threadIdx.x == 0) {
         for (int i = 0; i < SC_STAGES; ++i) {
             mbar_init(&full[i], 1);
@@ -605,8 +609,8 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
         fence_mbar_init();
     }
     __syncthreads();
-    // ---- phase 1: stream -> ballot words + count ----
-    int64_t cnt = 0;
+    // ---- phase 1: stream -> ballot words + per-chunk counts ----
+    int cnt = 0;
     if (warp == SC_CW) {
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
@@ -616,12 +620,12 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
                 if (t >= SC_STAGES) mbar_wait(&empty[st], ph ^ 1u);
                 const int64_t r0 = (c0 + t * SC_CHUNKS) * 1024;
                 const int64_t r1 = min((c0 + (t + 1) * SC_CHUNKS) * 1024, c1 * 1024);
-                if (r1 <= n && ((r1 - r0) * (int64_t)sizeof(T)) % 16 == 0) {
-                    const uint32_t bytes = (uint32_t)((r1 - r0) * sizeof(T));
+                if (r1 <= n) {
+                    const uint32_t bytes = (uint32_t)((r1 - r0) * sizeof(T));  // whole chunks: a multiple of 16
                     mbar_expect_tx(&full[st], bytes);
                     tma_load_1d(smem + (size_t)st * TB, col + r0, bytes, &full[st], pol);
                 } else {
-                    mbar_arrive(&full[st]);  // the ragged end of the column: consumers load it directly
+                    mbar_arrive(&full[st]);  // the column's ragged end: consumers load it directly
                 }
                 if (++st == SC_STAGES) { st = 0; ph ^= 1u; }
             }
@@ -633,41 +637,44 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
         for (int64_t t = 0; t < ntile; ++t) {
             mbar_wait(&full[st], ph);
             const int64_t c = c0 + t * SC_CHUNKS + warp;  // this warp's chunk
-            const int64_t r0 = (c0 + t * SC_CHUNKS) * 1024;
-            const int64_t r1 = min((c0 + (t + 1) * SC_CHUNKS) * 1024, c1 * 1024);
-            const bool staged = r1 <= n && ((r1 - r0) * (int64_t)sizeof(T)) % 16 == 0;
+            const bool staged = min((c0 + (t + 1) * SC_CHUNKS) * 1024, c1 * 1024) <= n;
             uint32_t mine = 0;
             if (c < c1) {
-                const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
-#pragma unroll 8
-                for (int k = 0; k < 32; ++k) {
-                    const int64_t r = c * 1024 + k * 32 + lane;
-                    bool f;
-                    if (staged) {
+                if (staged) {
+                    const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
+#pragma unroll
+                    for (int k = 0; k < 32; ++k) {
                         const T v = src[k * 32 + lane];
-                        f = v >= lo && v <= hi;  // NaN / INT_MIN (epsilon) fail: bounds from the host
-                    } else {
-                        f = false;
+                        const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
+                        mine = lane == k ? b : mine;
+                    }
+                } else {
+                    for (int k = 0; k < 32; ++k) {
+                        const int64_t r = c * 1024 + k * 32 + lane;
+                        bool f = false;
                         if (r < n) {
                             const T v = __ldg(col + r);
                             f = v >= lo && v <= hi;
                         }
+                        const uint32_t b = __ballot_sync(VD_FULL, f);
+                        mine = lane == k ? b : mine;
                     }
-                    const uint32_t b = __ballot_sync(VD_FULL, f);
-                    if (lane == k) mine = b;
                 }
-                bits[c * 32 + lane] = mine;
-                cnt += __popc(mine);
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(&empty[st]);
             if (++st == SC_STAGES) { st = 0; ph ^= 1u; }
+            if (c < c1) {
+                bits[c * 32 + lane] = mine;
+                int cc = __popc(mine);
+#pragma unroll
+                for (int o = 16; o; o >>= 1) cc += __shfl_xor_sync(VD_FULL, cc, o);
+                if (lane == 0) s_ccnt[c - c0] = (uint16_t)cc;
+                cnt += cc;
+            }
         }
     }
-    // CTA count -> counts[cta]
-#pragma unroll
-    for (int o = 16; o; o >>= 1) cnt += __shfl_xor_sync(VD_FULL, cnt, o);
-    if (lane == 0 && warp < SC_CW) s_cnt[warp] = (int)cnt;
+    if (lane == 0 && warp < SC_CW) s_cnt[warp] = cnt;
     __syncthreads();
     if (threadIdx.x == 0) {
         int64_t t = 0;
@@ -682,7 +689,8 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     // CTA base = counts of the CTAs before it
     if (warp == 0) {
         int64_t b = 0;
-        for (int i = lane; i < (int)blockIdx.x; i += 32) b += (int64_t)ld_acquire_u64(reinterpret_cast<uint64_t*>(&counts[i]));
+        for (int i = lane; i < (int)blockIdx.x; i += 32)
+            b += (int64_t)ld_acquire_u64(reinterpret_cast<uint64_t*>(&counts[i]));
         b = warp_sum_i64(b);
         if (lane == 0) {
             s_base = b;
@@ -693,48 +701,62 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
         }
     }
+    // exclusive scan of the chunk counts -> int32 chunk offsets within the
+    // CTA (in the ring's memory, free now): thread i owns a contiguous run
+    int32_t* s_off = reinterpret_cast<int32_t*>(smem) + SC_CW * SC_STG;
+    const int per = (nch + SC_THREADS - 1) / SC_THREADS;
+    const int i0 = min(nch, (int)threadIdx.x * per), i1 = min(nch, i0 + per);
+    int mysum = 0;
+    for (int i = i0; i < i1; ++i) mysum += s_ccnt[i];
+    int incl = mysum;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        const int u = __shfl_up_sync(VD_FULL, incl, o);
+        if (lane >= o) incl += u;
+    }
+    if (lane == 31) s_scan[warp] = incl;
     __syncthreads();
-    // ---- phase 2: bitmap words -> positions ----
+    int wbase = 0;
+    for (int w = 0; w < warp; ++w) wbase += s_scan[w];
+    int run = wbase + incl - mysum;
+    for (int i = i0; i < i1; ++i) {
+        s_off[i] = run;
+        run += s_ccnt[i];
+    }
+    __syncthreads();
+    // ---- phase 2: bitmap words -> positions, chunk by chunk, no barriers ----
     if (warp == SC_CW) return;
     const unsigned lt = lanemask_lt();
     int32_t* sw = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
-    int64_t run = s_base;
-    for (int64_t t = 0; t < ntile; ++t) {
-        const int64_t c = c0 + t * SC_CHUNKS + warp;
-        const uint32_t word = c < c1 ? __ldcs(&bits[c * 32 + lane]) : 0u;
-        const int wc = __popc(word);
-        int tot = wc;
+    const int64_t base = s_base;
+    // next non-empty chunk of this warp at or after index i (stride SC_CW)
+    auto next_nz = [&](int i) {
+        while (i < nch && s_ccnt[i] == 0) i += SC_CW;
+        return i;
+    };
+    int i = next_nz(warp);
+    uint32_t word = i < nch ? __ldcs(&bits[(c0 + i) * 32 + lane]) : 0u;
+    while (i < nch) {
+        const int inext = next_nz(i + SC_CW);
+        const uint32_t wnext = inext < nch ? __ldcs(&bits[(c0 + inext) * 32 + lane]) : 0u;  // in flight
+        uint32_t bw[32];
 #pragma unroll
-        for (int o = 16; o; o >>= 1) tot += __shfl_xor_sync(VD_FULL, tot, o);
-        if (lane == 0) s_cnt[warp] = tot;
-        bar_sync_n(1, SC_CW * 32);
-        int woff = 0, ttot = 0;
-#pragma unroll
-        for (int w = 0; w < SC_CW; ++w) {
-            const int x = s_cnt[w];
-            woff += w < warp ? x : 0;
-            ttot += x;
-        }
-        bar_sync_n(1, SC_CW * 32);  // s_cnt is rewritten next tile
-        if (c < c1 && tot > 0) {
-            uint32_t bw[32];
-#pragma unroll
-            for (int k = 0; k < 32; ++k) bw[k] = __shfl_sync(VD_FULL, word, k);
-            const int64_t g0 = run + woff;
-            const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
-            const int total = sc_stage_positions<MODE>(bw, c * 1024, a, sw, lane, lt);
-            __syncwarp();
-            sc_flush(sw, a, total, out + g0 - a, lane);
-            __syncwarp();
-        }
-        run += ttot;
+        for (int k = 0; k < 32; ++k) bw[k] = __shfl_sync(VD_FULL, word, k);
+        const int64_t g0 = base + s_off[i];
+        const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+        const int total = sc_stage_positions<MODE>(bw, (c0 + i) * 1024, a, sw, lane, lt);
+        __syncwarp();
+        sc_flush(sw, a, total, out + g0 - a, lane);
+        __syncwarp();
+        i = inext;
+        word = wnext;
     }
 }
 
 static size_t sel_coop_smem(size_t tsize) {
-    const size_t ring = (size_t)SC_STAGES * SC_CHUNKS * 1024 * tsize + 2 * SC_STAGES * 8;
-    const size_t stg = (size_t)SC_CW * SC_STG * 4;
-    return ring > stg ? ring : stg;
+    const size_t ring = (size_t)SC_STAGES * SC_CHUNKS * 1024 * tsize;
+    const size_t p2 = (size_t)SC_CW * SC_STG * 4 + (size_t)SC_MAXCH * 4;  // stages + chunk offsets
+    return std::max(ring, p2) + 2 * SC_STAGES * 8 + (size_t)SC_MAXCH * 2;
 }
 
 // VD_SELECT_COOP=0 keeps the 4-launch bitmap path (comparison runs)
@@ -762,6 +784,7 @@ static cudaError_t run_select_coop(const T* col, T lo, T hi, int64_t n, int32_t*
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SC_THREADS, sm) != cudaSuccess || per_sm < 1)
         return cudaErrorCooperativeLaunchTooLarge;
     int grid = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, std::min<int64_t>(nchunks, 4096));
+    if ((nchunks + grid - 1) / grid > SC_MAXCH) return cudaErrorNotSupported;  // caller falls back
     cudaError_t e = cudaMemsetAsync(bar, 0, 4, s);
     if (e != cudaSuccess) return e;
     void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&out_pos, (void*)&out_count,
@@ -1047,8 +1070,10 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         if constexpr (sizeof(T) == 4) {
-            if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0)
-                return run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+            if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0) {
+                cudaError_t e = run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+                if (e != cudaErrorNotSupported) return e;  // else: more chunks per CTA than fit, bitmap path
+            }
         }
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L) {

@@ -55,6 +55,57 @@ __device__ __forceinline__ int4 ld_stream16(const void* p) {
                  : "l"(p));
     return r;
 }
+// Isolated (late / random) loads: by default an L1 miss fetches the whole
+// 128-byte line from DRAM (scripts/ubench_dram_gran.cu: 125 B of DRAM per
+// random 4-byte load); the .L2::64B prefetch size makes it one 64-byte block
+// (63 B per load) -- the granule of the algorithmic byte models A31 / A33.
+__device__ __forceinline__ uint32_t ld64b_u8(const void* p) {
+    uint16_t v;
+    asm volatile("ld.global.nc.L2::64B.u8 %0, [%1];" : "=h"(v) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ uint32_t ld64b_u32(const void* p) {
+    uint32_t v;
+    asm volatile("ld.global.nc.L2::64B.u32 %0, [%1];" : "=r"(v) : "l"(p));
+    return v;
+}
+__device__ __forceinline__ uint64_t ld64b_u64(const void* p) {
+    uint64_t v;
+    asm volatile("ld.global.nc.L2::64B.u64 %0, [%1];" : "=l"(v) : "l"(p));
+    return v;
+}
+template <typename T>
+__device__ __forceinline__ T ldg64b(const T* p) {
+    static_assert(sizeof(T) == 1 || sizeof(T) == 4 || sizeof(T) == 8, "1-, 4- or 8-byte element");
+    T v;
+    if (sizeof(T) == 1) { const uint8_t x = (uint8_t)ld64b_u8(p); memcpy(&v, &x, 1); }
+    else if (sizeof(T) == 4) { const uint32_t x = ld64b_u32(p); memcpy(&v, &x, 4); }
+    else { const uint64_t x = ld64b_u64(p); memcpy(&v, &x, 8); }
+    return v;
+}
+// 128-bit streaming load with an L2 eviction-policy hint (evict_first for a
+// single-use scan, so it does not push out a table other rows update)
+__device__ __forceinline__ int4 ld_stream16_hint(const void* p, uint64_t pol) {
+    int4 r;
+    asm volatile("ld.global.nc.L1::no_allocate.L2::cache_hint.v4.s32 {%0,%1,%2,%3}, [%4], %5;"
+                 : "=r"(r.x), "=r"(r.y), "=r"(r.z), "=r"(r.w)
+                 : "l"(p), "l"(pol));
+    return r;
+}
+// global reductions with an L2 eviction-policy hint (evict_last: a grouping
+// table that must stay L2-resident under a streaming scan)
+__device__ __forceinline__ void red_add_u64_hint(unsigned long long* p, unsigned long long v, uint64_t pol) {
+    asm volatile("red.relaxed.gpu.global.add.L2::cache_hint.u64 [%0], %1, %2;" ::"l"(p), "l"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void red_add_f64_hint(double* p, double v, uint64_t pol) {
+    asm volatile("red.relaxed.gpu.global.add.L2::cache_hint.f64 [%0], %1, %2;" ::"l"(p), "d"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void red_min_s64_hint(long long* p, long long v, uint64_t pol) {
+    asm volatile("red.relaxed.gpu.global.min.L2::cache_hint.s64 [%0], %1, %2;" ::"l"(p), "l"(v), "l"(pol) : "memory");
+}
+__device__ __forceinline__ void red_max_s64_hint(long long* p, long long v, uint64_t pol) {
+    asm volatile("red.relaxed.gpu.global.max.L2::cache_hint.s64 [%0], %1, %2;" ::"l"(p), "l"(v), "l"(pol) : "memory");
+}
 __device__ __forceinline__ int2 ld_stream8(const void* p) {
     int2 r;
     asm volatile("ld.global.nc.L1::no_allocate.v2.s32 {%0,%1}, [%2];" : "=r"(r.x), "=r"(r.y) : "l"(p));
@@ -71,13 +122,15 @@ __device__ __forceinline__ int ld_stream4(const void* p) {
 // inline-PTX block: every address is ready before the first load issues, so
 // all eight are in flight together (left to itself the compiler consumes each
 // gather before computing the next address).
+// Eight predicated random loads issued back to back (memory-level
+// parallelism); each moves one 64-byte block (.L2::64B, see ld64b_*).
 __device__ __forceinline__ void gather8(const int64_t* const* p, const bool* pr, int64_t dflt, int64_t* v) {
-    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b64 %0, %24;\n\tmov.b64 %1, %24;\n\tmov.b64 %2, %24;\n\tmov.b64 %3, %24;\n\tmov.b64 %4, %24;\n\tmov.b64 %5, %24;\n\tmov.b64 %6, %24;\n\tmov.b64 %7, %24;\n\t@q0 ld.global.nc.b64 %0, [%8];\n\t@q1 ld.global.nc.b64 %1, [%9];\n\t@q2 ld.global.nc.b64 %2, [%10];\n\t@q3 ld.global.nc.b64 %3, [%11];\n\t@q4 ld.global.nc.b64 %4, [%12];\n\t@q5 ld.global.nc.b64 %5, [%13];\n\t@q6 ld.global.nc.b64 %6, [%14];\n\t@q7 ld.global.nc.b64 %7, [%15];\n\t}"
+    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b64 %0, %24;\n\tmov.b64 %1, %24;\n\tmov.b64 %2, %24;\n\tmov.b64 %3, %24;\n\tmov.b64 %4, %24;\n\tmov.b64 %5, %24;\n\tmov.b64 %6, %24;\n\tmov.b64 %7, %24;\n\t@q0 ld.global.nc.L2::64B.b64 %0, [%8];\n\t@q1 ld.global.nc.L2::64B.b64 %1, [%9];\n\t@q2 ld.global.nc.L2::64B.b64 %2, [%10];\n\t@q3 ld.global.nc.L2::64B.b64 %3, [%11];\n\t@q4 ld.global.nc.L2::64B.b64 %4, [%12];\n\t@q5 ld.global.nc.L2::64B.b64 %5, [%13];\n\t@q6 ld.global.nc.L2::64B.b64 %6, [%14];\n\t@q7 ld.global.nc.L2::64B.b64 %7, [%15];\n\t}"
                  : "=l"(v[0]), "=l"(v[1]), "=l"(v[2]), "=l"(v[3]), "=l"(v[4]), "=l"(v[5]), "=l"(v[6]), "=l"(v[7])
                  : "l"(p[0]), "l"(p[1]), "l"(p[2]), "l"(p[3]), "l"(p[4]), "l"(p[5]), "l"(p[6]), "l"(p[7]), "r"((int)pr[0]), "r"((int)pr[1]), "r"((int)pr[2]), "r"((int)pr[3]), "r"((int)pr[4]), "r"((int)pr[5]), "r"((int)pr[6]), "r"((int)pr[7]), "l"(dflt));
 }
 __device__ __forceinline__ void gather8(const int32_t* const* p, const bool* pr, int32_t dflt, int32_t* v) {
-    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b32 %0, %24;\n\tmov.b32 %1, %24;\n\tmov.b32 %2, %24;\n\tmov.b32 %3, %24;\n\tmov.b32 %4, %24;\n\tmov.b32 %5, %24;\n\tmov.b32 %6, %24;\n\tmov.b32 %7, %24;\n\t@q0 ld.global.nc.b32 %0, [%8];\n\t@q1 ld.global.nc.b32 %1, [%9];\n\t@q2 ld.global.nc.b32 %2, [%10];\n\t@q3 ld.global.nc.b32 %3, [%11];\n\t@q4 ld.global.nc.b32 %4, [%12];\n\t@q5 ld.global.nc.b32 %5, [%13];\n\t@q6 ld.global.nc.b32 %6, [%14];\n\t@q7 ld.global.nc.b32 %7, [%15];\n\t}"
+    asm volatile("{\n\t.reg .pred q<8>;\n\tsetp.ne.b32 q0, %16, 0;\n\tsetp.ne.b32 q1, %17, 0;\n\tsetp.ne.b32 q2, %18, 0;\n\tsetp.ne.b32 q3, %19, 0;\n\tsetp.ne.b32 q4, %20, 0;\n\tsetp.ne.b32 q5, %21, 0;\n\tsetp.ne.b32 q6, %22, 0;\n\tsetp.ne.b32 q7, %23, 0;\n\tmov.b32 %0, %24;\n\tmov.b32 %1, %24;\n\tmov.b32 %2, %24;\n\tmov.b32 %3, %24;\n\tmov.b32 %4, %24;\n\tmov.b32 %5, %24;\n\tmov.b32 %6, %24;\n\tmov.b32 %7, %24;\n\t@q0 ld.global.nc.L2::64B.b32 %0, [%8];\n\t@q1 ld.global.nc.L2::64B.b32 %1, [%9];\n\t@q2 ld.global.nc.L2::64B.b32 %2, [%10];\n\t@q3 ld.global.nc.L2::64B.b32 %3, [%11];\n\t@q4 ld.global.nc.L2::64B.b32 %4, [%12];\n\t@q5 ld.global.nc.L2::64B.b32 %5, [%13];\n\t@q6 ld.global.nc.L2::64B.b32 %6, [%14];\n\t@q7 ld.global.nc.L2::64B.b32 %7, [%15];\n\t}"
                  : "=r"(v[0]), "=r"(v[1]), "=r"(v[2]), "=r"(v[3]), "=r"(v[4]), "=r"(v[5]), "=r"(v[6]), "=r"(v[7])
                  : "l"(p[0]), "l"(p[1]), "l"(p[2]), "l"(p[3]), "l"(p[4]), "l"(p[5]), "l"(p[6]), "l"(p[7]), "r"((int)pr[0]), "r"((int)pr[1]), "r"((int)pr[2]), "r"((int)pr[3]), "r"((int)pr[4]), "r"((int)pr[5]), "r"((int)pr[6]), "r"((int)pr[7]), "r"(dflt));
 }
@@ -205,6 +258,12 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
         : "memory");
 }
 // L2 eviction policy for single-use streaming data.
+// L2 eviction policy for data re-read by other rows (lookups, group tables).
+__device__ __forceinline__ uint64_t policy_evict_last() {
+    uint64_t p;
+    asm volatile("createpolicy.fractional.L2::evict_last.b64 %0, 1.0;" : "=l"(p));
+    return p;
+}
 __device__ __forceinline__ uint64_t policy_evict_first() {
     uint64_t p;
     asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(p));

@@ -55,6 +55,23 @@ __device__ __forceinline__ Val fetch_typed(const void* p, int32_t dt, int64_t ro
     return v;
 }
 
+// The same, for an isolated (late / random) row: the load moves one 64-byte
+// block, not the default 128-byte line (ld64b_*, vd_common.cuh).
+__device__ __forceinline__ Val fetch_typed_64b(const void* p, int32_t dt, int64_t row) {
+    Val v;
+    v.isf = false;
+    v.i = 0;
+    v.f = 0;
+    switch (dt) {
+    case VD_U8: { uint8_t x = (uint8_t)ld64b_u8((const uint8_t*)p + row); v.eps = Eps<uint8_t>::is(x); v.i = x; break; }
+    case VD_I32: { int32_t x = (int32_t)ld64b_u32((const int32_t*)p + row); v.eps = Eps<int32_t>::is(x); v.i = x; break; }
+    case VD_I64: { int64_t x = (int64_t)ld64b_u64((const int64_t*)p + row); v.eps = Eps<int64_t>::is(x); v.i = x; break; }
+    case VD_F32: { float x = __uint_as_float(ld64b_u32((const float*)p + row)); v.eps = Eps<float>::is(x); v.isf = true; v.f = x; break; }
+    default: { double x = __longlong_as_double((long long)ld64b_u64((const double*)p + row)); v.eps = Eps<double>::is(x); v.isf = true; v.f = x; break; }
+    }
+    return v;
+}
+
 __device__ __forceinline__ bool term_true(const DevTerm& t, const Val& v) {
     if (v.eps) return false;  // a predicate on epsilon is "not selected" (reading A9)
     return v.isf ? cmp_flt(t.cmp, v.f, t.fv) : cmp_int(t.cmp, v.i, t.iv);
