@@ -470,9 +470,9 @@ def test_scatter_permutation_unique():
     v = gen.host(gen.F32_UNIFORM, n, seed=4)
     out = torch.empty(n, dtype=torch.float32, device="cuda")
     vd.scatter(vd.column(cuda_tensor(v)), cuda_tensor(pi), n, out, n, unique=True)
-    exp = np.empty(n, dtype=np.float32)
-    exp[pi] = v
-    assert np.array_equal(out.cpu().numpy(), exp)
+    po = oracle.run("o := Scatter(v, %d, p)" % n, v=v.astype(np.float64), p=pi.astype(np.int64))
+    exp = np.array(po.get("o"), dtype=np.float64)  # a permutation: every slot written (no epsilon)
+    assert np.array_equal(out.cpu().numpy().astype(np.float64), exp)
 
 
 @pytest.mark.parametrize("n,P", [(0, 4), (10, 4), (4097, 6), (300001, 175), (70000, 1024)])
@@ -499,25 +499,30 @@ def test_partition_vs_interpreter(n, P):
 def test_select_flag_pass_tiles_and_tail(mode, dtype, offset):
     """Several 16384-row tiles of the TMA flag pass plus a ragged LDG tail; a
     base pointer 4 bytes past a 16-byte boundary takes the LDG pass instead.
-    Positions must equal flatnonzero of the predicate either way."""
+    Positions must equal the interpreter's FoldSelect of the predicate
+    (P:L101-108)."""
     n = 5 * 16384 + 1000 + 7
     rng = np.random.default_rng(99)
     if dtype == "u8":
         a = rng.integers(0, 255, n + 16).astype(np.uint8)  # 0xFF = epsilon excluded by the interval
         op, c = ">", 100
-        ref = (a > 100) & (a != 0xFF)
+        prog = "p := Greater(v, 100)"
     elif dtype == "i32":
         a = rng.integers(-1000, 1000, n + 16).astype(np.int32)
         op, c = "<=", 17
-        ref = a <= 17
+        prog = "p := Greater(18, v)"
     else:
         a = rng.random(n + 16).astype(np.float32)
         op, c = "<", 0.25
-        ref = a < np.float32(0.25)
+        prog = "p := Greater(%s, v)" % float(np.float32(0.25)).hex()
+    eps = (a == 0xFF) if dtype == "u8" else np.zeros(a.size, bool)
     esz = a.itemsize
     skip = offset // esz
     da = cuda_tensor(a)[skip:skip + n]
-    exp = np.flatnonzero(ref[skip:skip + n])
+    w = a[skip:skip + n]
+    vals = w.astype(np.float64) if dtype == "f32" else w.astype(np.int64)
+    po = oracle.run(prog + "\npos := FoldSelect(p)", v=(vals, eps[skip:skip + n]))
+    exp = np.array([x for x in po.get("pos") if x is not None], dtype=np.int64)
     out = torch.empty(n, dtype=torch.int32, device="cuda")
     cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
     fn = vd.select_branch if mode == "branch" else vd.select_predicated

@@ -411,7 +411,9 @@ def test_fkj_q9_epsilon_vs_interpreter(variant):
 
 
 def test_generic_min_max_and_float_products():
-    """Generic fragment: MIN/MAX and float aggregates, grouped, with epsilon."""
+    """Generic fragment: MIN/MAX and float aggregates, grouped, with epsilon;
+    against the interpreter's Fig 10/11 program (FoldSelect -> Gather ->
+    Partition -> Scatter -> FoldMin / FoldMax / FoldSum / FoldCount)."""
     n = 200003
     rng = np.random.default_rng(1)
     k = rng.integers(0, 5, n).astype(np.int32)
@@ -422,15 +424,46 @@ def test_generic_min_max_and_float_products():
     plan = vd.pipeline(pred_=vd.pred([[(1, ">", -5 * 10**8)]]), key=[(0, 0, 0, 1)], ngroups=5,
                        aggs=[("min", [1]), ("max", [1]), ("sum", [2, (1, 0, 1)]), ("sum", [(2, 1, 2)]), ("count",)])
     got = vd.decode_partials(run(plan, views, n)[0], plan, float_aggs=[False, False, True, True, False])
-    m = x > -5 * 10**8  # epsilon never passes a predicate (A9)
-    for g in range(5):
-        s = m & (k == g)
-        assert got[g][0] == int(x[s].min()) and got[g][1] == int(x[s].max())
-        ref = float(np.sum(f[s] * x[s].astype(np.float64)))
-        assert abs(got[g][2] - ref) <= 1e-9 * abs(ref)
-        ref2 = float(np.sum(1 + 2 * f[s]))
-        assert abs(got[g][3] - ref2) <= 1e-9 * abs(ref2)
-        assert got[g][4] == int(s.sum()) == got[g][5]
+    ex = x == -2**63
+    p = oracle.Program()
+    p.set("t.k", k)
+    p.set("t.x", np.where(ex, 0, x), ex)
+    p.set("t.f", f)
+    p.run("""
+keep := Greater(t.x, -500000000)
+positions := FoldSelect(keep)
+sel := Gather(t, positions)
+fx := Multiply(sel.f, sel.x)
+f2 := Multiply(sel.f, 2)
+g2 := Add(f2, 1)
+vals := Zip(sel.k, sel.x, fx, g2)
+pivot := Range(0, 5, 1)
+ppos := Partition(sel.k, pivot)
+sc := Scatter(vals, vals, ppos)
+mn := FoldMin(sc.k, sc.x)
+mx := FoldMax(sc.k, sc.x)
+s1 := FoldSum(sc.k, sc.fx)
+s2 := FoldSum(sc.k, sc.g2)
+cnt := FoldCount(sc.k, sc.k)
+gk := FoldMax(sc.k, sc.k)
+gpos := FoldSelect(cnt)
+o_k := Gather(gk, gpos)
+o_mn := Gather(mn, gpos)
+o_mx := Gather(mx, gpos)
+o_s1 := Gather(s1, gpos)
+o_s2 := Gather(s2, gpos)
+o_c := Gather(cnt, gpos)
+""")
+    keys = p.get("o_k")
+    outs = {o: p.get(o) for o in ("o_mn", "o_mx", "o_s1", "o_s2", "o_c")}
+    exp = {kk: [outs[o][j] for o in ("o_mn", "o_mx", "o_s1", "o_s2", "o_c")] for j, kk in enumerate(keys)
+           if kk is not None}
+    assert set(got) == set(exp)
+    for g, e in exp.items():
+        assert got[g][0] == e[0] and got[g][1] == e[1]
+        assert abs(got[g][2] - e[2]) <= 1e-9 * abs(e[2])
+        assert abs(got[g][3] - e[3]) <= 1e-9 * abs(e[3])
+        assert got[g][4] == e[4] == got[g][5]
 
 
 def test_virtual_shards_merge_equals_whole_q1():
@@ -643,7 +676,9 @@ def test_late_fragment_selectivity_estimate():
 def test_late_fragment_edge_sizes(n, lead):
     """Late fragment at sizes around its 16-row lead words and 32-row drains
     (tail rows only, one word, one word + tail, partial drains) with leads
-    that pass nothing, everything or some rows; against numpy."""
+    that pass nothing, everything or some rows; against the interpreter
+    (FoldSelect of the lead and the gathered dimension term, Gather,
+    FoldSum / FoldCount)."""
     rng = np.random.default_rng(n * 7 + len(lead))
     m = 300
     a = rng.integers(0, 4, n).astype(np.uint8)
@@ -653,9 +688,24 @@ def test_late_fragment_edge_sizes(n, lead):
     cmp_, val = {"none": ("==", 9), "all": ("<=", 3), "some": ("==", 2)}[lead]
     plan = vd.pipeline(pred_=vd.pred([[(0, cmp_, val), (3, "<", 5)]]), gathers=[(1, 0, 1)],
                        aggs=[("sum", [2]), ("count",)])
-    lead_ok = (a == val) if cmp_ == "==" else (a <= val)
-    sel = lead_ok & (d[fk - 1] < 5)
-    exp = {0: [int(x[sel].sum()), int(sel.sum()), int(sel.sum())]} if sel.any() else {}
+    lead_term = "c1 := Equals(f.a, %d)" % val if cmp_ == "==" else "c1 := Greater(%d, f.a)" % (val + 1)
+    p = oracle.Program()
+    p.set("f.a", a)
+    p.set("f.fk", fk)
+    p.set("f.x", x)
+    p.set("dim.d", d)
+    p.run(lead_term + """
+pk := Subtract(f.fk, 1)
+dd := Gather(dim.d, pk)
+c2 := Greater(5, dd)
+keep := LogicalAnd(c1, c2)
+positions := FoldSelect(keep)
+sel := Gather(f.x, positions)
+total := FoldSum(sel)
+cnt := FoldCount(positions)
+""")
+    c = p.get("cnt")[0] if n else 0
+    exp = {0: [p.get("total")[0], c, c]} if c else {}
     keep, views = load([a, fk, x])
     dkeep, dviews = load([d])
     with env(VD_LATE="force"):
