@@ -153,6 +153,161 @@ __device__ __forceinline__ int64_t hg_global_slot(const HgArgs& a, int64_t key) 
     return -1;
 }
 
+// Fold one row's words (v[ag], has[ag]; the row count is word naggs) into
+// the CTA's shared table, or spill to the global one.  Once the shared table
+// is 3/4 full a new key gets only 2 probes there: with uniform keys over a
+// large domain a CTA sees few repeats, and probing a full table only adds
+// latency.
+__device__ __forceinline__ void hg_insert(const HgArgs& a, long long* s_key, unsigned long long* s_val,
+                                          int* s_used, int64_t key, const unsigned long long* v, const bool* has,
+                                          uint64_t pol_t) {
+    const int W = a.naggs + 1;
+    uint32_t h = (uint32_t)(hg_mix(key) & (HG_SLOTS - 1));
+    const int probes = *((volatile int*)s_used) < HG_SLOTS * 3 / 4 ? HG_PROBES : 2;
+    int slot = -1;
+    for (int p = 0; p < probes; ++p) {
+        const long long cur = s_key[h];
+        if (cur == key) { slot = (int)h; break; }
+        if (cur == HG_EMPTY) {
+            const long long prev = (long long)atomicCAS((unsigned long long*)&s_key[h], (unsigned long long)HG_EMPTY,
+                                                        (unsigned long long)key);
+            if (prev == HG_EMPTY) { atomicAdd(s_used, 1); slot = (int)h; break; }
+            if (prev == key) { slot = (int)h; break; }
+        }
+        h = (h + 1) & (HG_SLOTS - 1);
+    }
+    if (slot >= 0) {
+        unsigned long long* dst = s_val + (size_t)slot * W;
+        for (int ag = 0; ag <= a.naggs; ++ag)
+            if (has[ag]) hg_atomic(dst + ag, ag < a.naggs ? a.kind[ag] : VD_AGG_COUNT, ag < a.naggs ? a.isf[ag] : 0, v[ag]);
+        return;
+    }
+    const int64_t g = hg_global_slot(a, key);  // level 2: spill to the global table
+    if (g < 0) return;
+    unsigned long long* dst = a.vals + (size_t)g * W;
+    for (int ag = 0; ag <= a.naggs; ++ag) {
+        if (!has[ag]) continue;
+        const int kind = ag < a.naggs ? a.kind[ag] : VD_AGG_COUNT;
+        const int fl = ag < a.naggs ? a.isf[ag] : 0;
+        if (kind == VD_AGG_SUM && fl) red_add_f64_hint((double*)(dst + ag), __longlong_as_double((long long)v[ag]), pol_t);
+        else if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) red_add_u64_hint(dst + ag, v[ag], pol_t);
+        else if (kind == VD_AGG_MIN) red_min_s64_hint((long long*)(dst + ag), (long long)v[ag], pol_t);
+        else red_max_s64_hint((long long*)(dst + ag), (long long)v[ag], pol_t);
+    }
+}
+
+// flush the CTA's shared table into the global one
+__device__ __forceinline__ void hg_flush(const HgArgs& a, const long long* s_key, const unsigned long long* s_val) {
+    const int W = a.naggs + 1;
+    for (int k = threadIdx.x; k < HG_SLOTS; k += HG_THREADS) {
+        const long long key = s_key[k];
+        if (key == HG_EMPTY) continue;
+        const int64_t g = hg_global_slot(a, key);
+        if (g < 0) continue;
+        for (int ag = 0; ag <= a.naggs; ++ag) {
+            const int kind = ag < a.naggs ? a.kind[ag] : VD_AGG_COUNT;
+            const unsigned long long x = s_val[(size_t)k * W + ag];
+            if (x == hg_identity(kind) && kind != VD_AGG_SUM && kind != VD_AGG_COUNT) continue;
+            hg_atomic(a.vals + (size_t)g * W + ag, kind, ag < a.naggs ? a.isf[ag] : 0, x);
+        }
+    }
+}
+
+// Interval fast path (the predicate is one conjunction of integer interval
+// terms on at most two columns, the first 16-byte aligned -- Q15's
+// l_shipdate window): 4 rows per thread per 128-bit evict-first load of the
+// filter column, qualifying rows compacted per warp into a shared-memory
+// queue and folded 32 at a time with every lane busy (key, values and the
+// second filter column loaded late, 64-byte blocks).
+struct HgIv {
+    const void* c0;
+    const void* c1;  // nullptr: no second filter column
+    int32_t dt0, dt1;
+    int64_t lo0, hi0, lo1, hi1;
+};
+constexpr int HG_QCAP = 32 + 4 * 32;
+
+__global__ void __launch_bounds__(HG_THREADS) k_hg_fold_iv(const __grid_constant__ HgArgs a,
+                                                          const __grid_constant__ HgIv iv) {
+    extern __shared__ __align__(16) unsigned long long s_tab[];
+    __shared__ int64_t s_q[HG_THREADS / 32][HG_QCAP];
+    __shared__ int s_used;
+    const int W = a.naggs + 1;
+    long long* s_key = (long long*)s_tab;
+    unsigned long long* s_val = s_tab + HG_SLOTS;
+    for (int k = threadIdx.x; k < HG_SLOTS; k += HG_THREADS) s_key[k] = HG_EMPTY;
+    for (int k = threadIdx.x; k < HG_SLOTS * W; k += HG_THREADS) {
+        const int ag = k % W;
+        s_val[k] = ag < a.naggs ? hg_identity(a.kind[ag]) : 0ull;
+    }
+    if (threadIdx.x == 0) s_used = 0;
+    __syncthreads();
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const uint64_t pol_t = policy_evict_last(), pol_s = policy_evict_first();
+    int64_t* q_ = s_q[warp];
+    int cnt = 0;
+    const unsigned lt = lanemask_lt();
+    auto fold_row = [&](int64_t row) {
+        if (iv.c1) {
+            const Val y = fetch_typed_64b(iv.c1, iv.dt1, row);
+            if (y.eps || y.i < iv.lo1 || y.i > iv.hi1) return;
+        }
+        const Val k = fetch_typed_64b(a.cols.p[a.key_col], a.cols.dt[a.key_col], row);
+        if (k.eps) return;  // epsilon key: no group (A9)
+        unsigned long long v[VD_MAX_AGGS + 1];
+        bool has[VD_MAX_AGGS + 1];
+        for (int ag = 0; ag < a.naggs; ++ag) {
+            if (a.kind[ag] == VD_AGG_COUNT) { v[ag] = 1; has[ag] = true; }
+            else has[ag] = hg_value(a, ag, row, &v[ag]);
+        }
+        v[a.naggs] = 1;
+        has[a.naggs] = true;
+        hg_insert(a, s_key, s_val, &s_used, k.i, v, has, pol_t);
+    };
+    auto drain = [&](int k) {  // fold the top k (<= 32) queued rows
+        __syncwarp();
+        if (lane < k) fold_row(q_[cnt - k + lane]);
+        cnt -= k;
+        __syncwarp();
+    };
+    const int64_t nq = a.n / 4;
+    const int64_t wstride = (int64_t)gridDim.x * HG_THREADS;
+    for (int64_t q0 = (int64_t)blockIdx.x * HG_THREADS + warp * 32; q0 < nq; q0 += wstride) {
+        const int64_t q = q0 + lane;
+        int64_t x[4] = {INT64_MIN, INT64_MIN, INT64_MIN, INT64_MIN};
+        if (q < nq) {
+            if (iv.dt0 == VD_I32) {
+                const int4 w = ld_stream16_hint((const int32_t*)iv.c0 + 4 * q, pol_s);
+                x[0] = w.x; x[1] = w.y; x[2] = w.z; x[3] = w.w;
+            } else {
+                const int4 w0 = ld_stream16_hint((const int64_t*)iv.c0 + 4 * q, pol_s);
+                const int4 w1 = ld_stream16_hint((const int64_t*)iv.c0 + 4 * q + 2, pol_s);
+                x[0] = (int64_t)((uint64_t)(uint32_t)w0.y << 32 | (uint32_t)w0.x);
+                x[1] = (int64_t)((uint64_t)(uint32_t)w0.w << 32 | (uint32_t)w0.z);
+                x[2] = (int64_t)((uint64_t)(uint32_t)w1.y << 32 | (uint32_t)w1.x);
+                x[3] = (int64_t)((uint64_t)(uint32_t)w1.w << 32 | (uint32_t)w1.z);
+            }
+        }
+#pragma unroll
+        for (int j = 0; j < 4; ++j) {
+            const bool pass = x[j] >= iv.lo0 && x[j] <= iv.hi0;
+            const unsigned b = __ballot_sync(VD_FULL, pass);
+            if (pass) q_[cnt + __popc(b & lt)] = 4 * q + j;
+            cnt += __popc(b);
+        }
+        while (cnt >= 32) drain(32);
+    }
+    if (cnt > 0) drain(cnt);
+    if (blockIdx.x == 0 && threadIdx.x == 0) {  // ragged tail (< 4 rows)
+        for (int64_t row = nq * 4; row < a.n; ++row) {
+            const Val x = fetch_typed(iv.c0, iv.dt0, row);
+            if (!(x.eps || x.i < iv.lo0 || x.i > iv.hi0)) fold_row(row);
+        }
+    }
+    __syncthreads();
+    hg_flush(a, s_key, s_val);
+}
+
 __global__ void __launch_bounds__(HG_THREADS) k_hg_fold(const __grid_constant__ HgArgs a) {
     extern __shared__ __align__(16) unsigned long long s_tab[];  // [HG_SLOTS] keys, then [HG_SLOTS][W] words
     const int W = a.naggs + 1;
@@ -484,7 +639,58 @@ cudaError_t launch_hash_group_fold(const DevCols& cols, const DevPred& pred, int
     const int sms = num_sms();
     k_hg_init<<<sms * 8, HG_THREADS, 0, s>>>(A);
     ++*nl;
-    if (n > 0) {
+    // interval fast path: one conjunction of integer interval terms on at most
+    // two columns, the first i32/i64 and 16-byte aligned
+    HgIv iv;
+    std::memset(&iv, 0, sizeof(iv));
+    bool fast = pred.nconj == 1 && pred.nterms[0] >= 1;
+    int fc[2] = {-1, -1};
+    int64_t lo[2] = {INT64_MIN + 1, INT64_MIN + 1}, hi[2] = {INT64_MAX, INT64_MAX};
+    for (int k = 0; fast && k < pred.nterms[0]; ++k) {
+        const DevTerm& t = pred.t[0][k];
+        const int slot = t.col == fc[0] ? 0 : (t.col == fc[1] ? 1 : (fc[0] < 0 ? 0 : (fc[1] < 0 ? 1 : -1)));
+        if (slot < 0 || (cols.dt[t.col] != VD_I32 && cols.dt[t.col] != VD_I64)) { fast = false; break; }
+        fc[slot] = t.col;
+        switch (t.cmp) {
+        case VD_CMP_GT: if (t.iv == INT64_MAX) fast = false; else lo[slot] = std::max(lo[slot], t.iv + 1); break;
+        case VD_CMP_GE: lo[slot] = std::max(lo[slot], t.iv); break;
+        case VD_CMP_LT: if (t.iv == INT64_MIN) fast = false; else hi[slot] = std::min(hi[slot], t.iv - 1); break;
+        case VD_CMP_LE: hi[slot] = std::min(hi[slot], t.iv); break;
+        case VD_CMP_EQ: lo[slot] = std::max(lo[slot], t.iv); hi[slot] = std::min(hi[slot], t.iv); break;
+        default: fast = false;
+        }
+    }
+    if (fast) {
+        for (int j = 0; j < 2; ++j) {  // epsilon (the type's minimum) outside the interval (A9)
+            if (fc[j] < 0) continue;
+            const int64_t eps = cols.dt[fc[j]] == VD_I32 ? (int64_t)INT32_MIN : INT64_MIN;
+            if (lo[j] <= eps) lo[j] = eps + 1;
+        }
+        fast = ((uintptr_t)cols.p[fc[0]] % 16) == 0 && !getenv("VD_HASH_GENERIC");
+    }
+    if (n > 0 && fast) {
+        iv.c0 = cols.p[fc[0]];
+        iv.dt0 = cols.dt[fc[0]];
+        iv.lo0 = lo[0];
+        iv.hi0 = hi[0];
+        if (fc[1] >= 0) {
+            iv.c1 = cols.p[fc[1]];
+            iv.dt1 = cols.dt[fc[1]];
+            iv.lo1 = lo[1];
+            iv.hi1 = hi[1];
+        }
+        const size_t smem = (size_t)HG_SLOTS * 8 * (naggs + 2);
+        cudaFuncSetAttribute(k_hg_fold_iv, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        int per_sm = 0;
+        if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k_hg_fold_iv, HG_THREADS, smem) != cudaSuccess ||
+            per_sm < 1)
+            per_sm = 1;
+        const int64_t nq = n / 4;
+        const int grid = (int)std::max<int64_t>(
+            1, std::min<int64_t>((nq + HG_THREADS - 1) / HG_THREADS, (int64_t)sms * per_sm));
+        k_hg_fold_iv<<<grid, HG_THREADS, smem, s>>>(A, iv);
+        ++*nl;
+    } else if (n > 0) {
         const size_t smem = (size_t)HG_SLOTS * 8 * (naggs + 2);
         cudaFuncSetAttribute(k_hg_fold, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         int per_sm = 0;

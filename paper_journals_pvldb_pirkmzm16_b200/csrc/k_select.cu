@@ -503,83 +503,31 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
 // One cooperative persistent kernel (one CTA per SM, all co-resident), each
 // CTA owning a contiguous range of 1024-row chunks:
 //   phase 1  a producer warp streams the CTA's rows through an SC_STAGES-deep
-//            TMA ring; consumer warp w turns 1024 rows into 32 ballots (bit L
-//            of ballot 32q'+j... each ballot is a row-ordered 32-bit word: bit
-//            L <-> row 32k + L of the chunk) and stores them as the chunk's
-//            32 bitmap words (the predicate materialised, Fig 8's break: n/8
-//            bytes, largely L2-resident) while counting; the CTA's count goes
-//            to counts[cta].
-//   barrier  one grid-wide barrier; the CTA's output base is the sum of the
-//            counts of the CTAs before it (148 values: no scan launch, no
-//            per-tile look-back chain).
-//   phase 2  the CTA decodes its bitmap in order with a running offset: per
-//            tile of SC_CW chunks, warp counts -> CTA prefix -> every warp
-//            stages its positions in shared memory (branching: qualifying
-//            lanes at their rank; predicated: cursor arithmetic, every row
-//            stored at the cursor, the cursor advanced by the predicate,
-//            P:L101-108) and streams the ascending run out with 16-byte
-//            stores.  The ring's shared memory is reused for the stages.
-// Replaces the 4-launch bitmap path (flag pass, scan, total, position pass):
-// the step pays the column read once, the bitmap's n/8 bytes twice (mostly
-// in L2) and the positions once.  A single-pass decoupled look-back variant
-// (a look-back per 64 KB tile) was measured at 5.8 ms for 1e9 rows: under a
-// full HBM stream one look-back costs several microseconds of L2 round trips,
-// far above a CTA's ~1.5 us per tile.
+//            TMA ring; consumer warp w turns its 1024-row chunk into 32
+//            ballots (ballot k: bit L <-> row 32k + L, a row-ordered word)
+//            and stores them as the chunk's 32 bitmap words -- the predicate
+//            materialised, Fig 8's break: n/8 bytes, largely L2-resident --
+//            and the chunk's count in shared memory;
+//   barrier  the CTA's total goes to counts[cta]; one grid-wide barrier; the
+//            CTA's output base is the sum of the counts of the CTAs before it
+//            (no scan launch, no per-tile look-back chain), and a CTA-wide
+//            scan of its chunk counts gives every chunk's offset;
+//   phase 2  warps decode their chunks independently (no barriers), skipping
+//            empty chunks and keeping the next chunks' words in flight.
+// Replaces the 4-launch bitmap path (flag pass, scan, total, position pass).
+// A single-pass decoupled look-back variant (one look-back per 64 KB tile)
+// was measured at 5.8 ms for 1e9 rows: under a full HBM stream a look-back
+// costs several microseconds of L2 round trips, far above a CTA's ~1.5 us
+// per tile.
 static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
 constexpr int SC_CW = 16;
 constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
 constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
-constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
+constexpr int SC_STG = 1024 + 32 + 8;        // per-warp position stage (ints, padded 1 per 32)
+constexpr int SC_PF = 4;                     // phase 2: chunks in flight per warp
+constexpr int SC_SPARSE = 64;                // phase 2: branching chunks this sparse store directly
 constexpr int SC_MAXCH = 12288;              // chunks per CTA (counts kept in shared memory)
-
-template <int MODE>
-__device__ __forceinline__ int sc_stage_positions(const uint32_t (&bw)[32], int64_t row0, int a, int32_t* sw,
-                                                  int lane, unsigned lt) {
-    // stage index a + k <-> output k of the chunk
-    int cur = a;
-#pragma unroll
-    for (int q = 0; q < 8; ++q) {
-        const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
-        int pre = cur;
-#pragma unroll
-        for (int j = 0; j < 4; ++j) {
-            const uint32_t w = bw[4 * q + j];
-            const int f = (w >> lane) & 1u;
-            const int r = __popc(w & lt);
-            const int32_t row = (int32_t)(row0 + (4 * q + j) * 32 + lane);
-            if (MODE == 0) {
-                if (f) sw[pre + r] = row;
-            } else {
-                // cursor arithmetic: unconditional store; rows that do not
-                // qualify land past the block's count and are overwritten
-                const int sel_before = pre - cur + r;
-                const int k = f ? pre + r : cur + cq + (j * 32 + lane - sel_before);
-                sw[k] = row;
-            }
-            pre += __popc(w);
-        }
-        cur += cq;
-    }
-    return cur - a;
-}
-
-__device__ __forceinline__ void sc_flush(const int32_t* sw, int a, int total, int32_t* __restrict__ ob, int lane) {
-    const int ngr = (a + total + 3) >> 2;
-    for (int v = lane; v < ngr; v += 32) {
-        const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
-        if (4 * v >= a && 4 * v + 4 <= a + total) {
-            __stcs(reinterpret_cast<int4*>(ob) + v, x);
-        } else {
-            const int32_t xs[4] = {x.x, x.y, x.z, x.w};
-#pragma unroll
-            for (int e = 0; e < 4; ++e) {
-                const int k = 4 * v + e;
-                if (k >= a && k < a + total) __stcs(ob + k, xs[e]);
-            }
-        }
-    }
-}
 
 template <int MODE, typename T>
 __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
@@ -725,31 +673,101 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     }
     __syncthreads();
     // ---- phase 2: bitmap words -> positions, chunk by chunk, no barriers ----
+    // Lane L owns word L of a chunk (rows 32L .. 32L+31): a warp popc-prefix
+    // gives every lane its output range.  Sparse chunks (branching, at most
+    // SC_SPARSE positions) store straight to global memory; denser chunks
+    // assemble in a padded shared-memory stage (index k at k + k/32: lanes
+    // 32 positions apart hit different banks) and stream out with 16-byte
+    // stores; predicated mode always uses the stage with cursor arithmetic
+    // (every row written, qualifying rows at the cursor).  Each warp keeps the
+    // words of its next SC_PF non-empty chunks in flight (a register queue):
+    // at low selectivity the pass is otherwise one L2 round trip per chunk.
     if (warp == SC_CW) return;
-    const unsigned lt = lanemask_lt();
-    int32_t* sw = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
+    int32_t* st = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
     const int64_t base = s_base;
-    // next non-empty chunk of this warp at or after index i (stride SC_CW)
-    auto next_nz = [&](int i) {
-        while (i < nch && s_ccnt[i] == 0) i += SC_CW;
-        return i;
-    };
-    int i = next_nz(warp);
-    uint32_t word = i < nch ? __ldcs(&bits[(c0 + i) * 32 + lane]) : 0u;
-    while (i < nch) {
-        const int inext = next_nz(i + SC_CW);
-        const uint32_t wnext = inext < nch ? __ldcs(&bits[(c0 + inext) * 32 + lane]) : 0u;  // in flight
-        uint32_t bw[32];
+    int qi[SC_PF];
+    uint32_t qw[SC_PF];
+    int nxt = warp;
 #pragma unroll
-        for (int k = 0; k < 32; ++k) bw[k] = __shfl_sync(VD_FULL, word, k);
+    for (int u = 0; u < SC_PF; ++u) {
+        while (nxt < nch && s_ccnt[nxt] == 0) nxt += SC_CW;
+        qi[u] = nxt;
+        qw[u] = nxt < nch ? __ldcs(&bits[(c0 + nxt) * 32 + lane]) : 0u;
+        if (nxt < nch) nxt += SC_CW;
+    }
+    while (qi[0] < nch) {
+        const int i = qi[0];
+        const uint32_t w = qw[0];
+#pragma unroll
+        for (int u = 0; u + 1 < SC_PF; ++u) {
+            qi[u] = qi[u + 1];
+            qw[u] = qw[u + 1];
+        }
+        while (nxt < nch && s_ccnt[nxt] == 0) nxt += SC_CW;
+        qi[SC_PF - 1] = nxt;
+        qw[SC_PF - 1] = nxt < nch ? __ldcs(&bits[(c0 + nxt) * 32 + lane]) : 0u;
+        if (nxt < nch) nxt += SC_CW;
+        const int pc = __popc(w);
+        int incl = pc;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            const int u = __shfl_up_sync(VD_FULL, incl, o);
+            if (lane >= o) incl += u;
+        }
+        const int excl = incl - pc;
+        const int total = s_ccnt[i];
         const int64_t g0 = base + s_off[i];
+        const int32_t row0 = (int32_t)((c0 + i) * 1024 + lane * 32);
+        if (MODE == 0 && total <= SC_SPARSE) {
+            uint32_t m = w;
+            int k = excl;
+            while (m) {
+                __stcs(&out[g0 + k], row0 + (__ffs(m) - 1));
+                ++k;
+                m &= m - 1;
+            }
+            continue;
+        }
+        // output index k sits at stage index j = k + a (a = the output's
+        // misalignment in words), physically j + j/32: 16-byte output groups
+        // are 4-word stage groups that never straddle a pad
         const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
-        const int total = sc_stage_positions<MODE>(bw, (c0 + i) * 1024, a, sw, lane, lt);
+        if (MODE == 0) {
+            uint32_t m = w;
+            int k = excl + a;
+            while (m) {
+                st[k + (k >> 5)] = row0 + (__ffs(m) - 1);
+                ++k;
+                m &= m - 1;
+            }
+        } else {
+            int sel = excl + a, unsel = total + (lane * 32 - excl) + a;
+#pragma unroll
+            for (int b = 0; b < 32; ++b) {
+                const int f = (w >> b) & 1u;
+                const int k = f ? sel : unsel;
+                st[k + (k >> 5)] = row0 + b;
+                sel += f;
+                unsel += 1 - f;
+            }
+        }
         __syncwarp();
-        sc_flush(sw, a, total, out + g0 - a, lane);
+        // flush: scalar stores up to the first 16-byte boundary of the output,
+        // one 128-bit streaming store per lane per 128 positions, scalar tail
+        const int h = min(total, (4 - a) & 3);
+        if (lane < h) __stcs(&out[g0 + lane], st[lane + a]);  // j < 32: no pad yet
+        const int nv = (total - h) >> 2;
+        int4* o4 = reinterpret_cast<int4*>(out + g0 + h);
+        for (int v = lane; v < nv; v += 32) {
+            const int j = h + a + 4 * v;  // a multiple of 4
+            const int32_t* g = st + j + (j >> 5);
+            __stcs(o4 + v, make_int4(g[0], g[1], g[2], g[3]));
+        }
+        for (int k = h + 4 * nv + lane; k < total; k += 32) {
+            const int j = k + a;
+            __stcs(&out[g0 + k], st[j + (j >> 5)]);
+        }
         __syncwarp();
-        i = inext;
-        word = wnext;
     }
 }
 
