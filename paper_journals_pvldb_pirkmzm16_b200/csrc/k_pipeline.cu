@@ -54,6 +54,57 @@ __device__ __forceinline__ void put_f64(Slot16* s, double v) {
 }
 __device__ __forceinline__ double get_f64(const Slot16& s) { return __longlong_as_double((long long)s.lo); }
 
+// The grid level of Fig 3's hierarchical fold, in the last CTA to finish
+// (Fragment 2 of Fig 8): slot k = the fold over the CTAs'
+// partials parts[b * nslots + k].  One warp per slot, lanes taking blocks
+// b = lane, lane + 32, ... -- independent L2 loads, one round trip -- then a
+// fixed shuffle tree (deterministic per launch shape).  A thread-per-slot
+// loop over the blocks is a chain of gridDim dependent L2 loads (~20 us at
+// 148 CTAs: most of a small step, C1).  Every warp of the CTA must call it.
+enum FoldKind { FK_I128_SUM = 0, FK_F64_SUM = 1, FK_I128_MIN = 2, FK_I128_MAX = 3, FK_F64_MIN = 4, FK_F64_MAX = 5 };
+template <class KindOf>
+__device__ __forceinline__ void fold_grid_parts(const Slot16* __restrict__ parts, int nslots, Slot16* dst,
+                                                KindOf kind_of) {
+    const int lane = threadIdx.x & 31, nw = blockDim.x >> 5;
+    const unsigned nb = gridDim.x;
+    for (int k = threadIdx.x >> 5; k < nslots; k += nw) {
+        const int kd = kind_of(k);
+        Slot16 r;
+        if (kd == FK_F64_SUM || kd == FK_F64_MIN || kd == FK_F64_MAX) {
+            double t = kd == FK_F64_MIN ? DBL_MAX : (kd == FK_F64_MAX ? -DBL_MAX : 0.0);
+            for (unsigned b = lane; b < nb; b += 32) {
+                const double x = __longlong_as_double((long long)__ldcg(&parts[(size_t)b * nslots + k].lo));
+                t = kd == FK_F64_SUM ? t + x : (kd == FK_F64_MIN ? fmin(t, x) : fmax(t, x));
+            }
+#pragma unroll
+            for (int o = 16; o; o >>= 1) {
+                const double u = __shfl_xor_sync(VD_FULL, t, o);
+                t = kd == FK_F64_SUM ? t + u : (kd == FK_F64_MIN ? fmin(t, u) : fmax(t, u));
+            }
+            put_f64(&r, t);
+        } else {
+            i128 t = kd == FK_I128_MIN ? (i128)INT64_MAX : (kd == FK_I128_MAX ? (i128)INT64_MIN : (i128)0);
+            for (unsigned b = lane; b < nb; b += 32) {
+                Slot16 x;
+                x.lo = __ldcg(&parts[(size_t)b * nslots + k].lo);
+                x.hi = __ldcg(&parts[(size_t)b * nslots + k].hi);
+                const i128 y = get_i128(x);
+                t = kd == FK_I128_SUM ? t + y : (kd == FK_I128_MIN ? (y < t ? y : t) : (y > t ? y : t));
+            }
+#pragma unroll
+            for (int o = 16; o; o >>= 1) {
+                const i128 u = shfl_xor_i128(t, o);
+                t = kd == FK_I128_SUM ? t + u : (kd == FK_I128_MIN ? (u < t ? u : t) : (u > t ? u : t));
+            }
+            put_i128(&r, t);
+        }
+        if (lane == 0) dst[k] = r;
+    }
+}
+struct FkI128Sum {
+    __device__ __forceinline__ int operator()(int) const { return FK_I128_SUM; }
+};
+
 // Maps from a fragment's raw result slots to the plan's [ngroups][naggs+1].
 struct Q1Map {
     int32_t naggs, ngroups;
@@ -359,29 +410,15 @@ __global__ void __launch_bounds__(GEN_THREADS) k_pipe_generic(const __grid_const
     __syncthreads();
     if (!s_last2) return;
     __threadfence();
-    for (int k = threadIdx.x; k < nslots; k += GEN_THREADS) {
-        int a = k % (NA + 1);
+    fold_grid_parts(block_parts, nslots, out, [&](int k) {
+        const int a = k % (NA + 1);
         const bool cnt = (a == NA);
         const int kind = cnt ? VD_AGG_COUNT : P.agg[a].kind;
         const bool isf = cnt ? false : P.agg[a].isf;
-        Slot16 r;
-        r.lo = __ldcg(&block_parts[k].lo);
-        r.hi = __ldcg(&block_parts[k].hi);
-        for (unsigned b = 1; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&block_parts[(size_t)b * nslots + k].lo);
-            x.hi = __ldcg(&block_parts[(size_t)b * nslots + k].hi);
-            if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) {
-                if (isf) put_f64(&r, get_f64(r) + get_f64(x)); else put_i128(&r, get_i128(r) + get_i128(x));
-            } else if (isf) {
-                put_f64(&r, kind == VD_AGG_MIN ? fmin(get_f64(r), get_f64(x)) : fmax(get_f64(r), get_f64(x)));
-            } else {
-                i128 p = get_i128(r), q = get_i128(x);
-                put_i128(&r, kind == VD_AGG_MIN ? (q < p ? q : p) : (q > p ? q : p));
-            }
-        }
-        out[k] = r;
-    }
+        if (kind == VD_AGG_SUM || kind == VD_AGG_COUNT) return isf ? (int)FK_F64_SUM : (int)FK_I128_SUM;
+        if (isf) return kind == VD_AGG_MIN ? (int)FK_F64_MIN : (int)FK_F64_MAX;
+        return kind == VD_AGG_MIN ? (int)FK_I128_MIN : (int)FK_I128_MAX;
+    });
 }
 
 // ============================================================================
@@ -583,16 +620,7 @@ __global__ void __launch_bounds__(Q1_THREADS, 2) k_pipe_q1(const __grid_constant
     if (!s_last) return;
     __threadfence();
     __shared__ Slot16 s_raw[G * 6];
-    if (threadIdx.x < G * 6) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
-            t += get_i128(x);
-        }
-        put_i128(&s_raw[threadIdx.x], t);
-    }
+    fold_grid_parts(parts, G * 6, s_raw, FkI128Sum());
     __syncthreads();
     // the plan's [ngroups][naggs+1] layout (slot naggs = row count = COUNT)
     for (int k = threadIdx.x; k < map.ngroups * (map.naggs + 1); k += blockDim.x) {
@@ -756,16 +784,7 @@ __global__ void __launch_bounds__(Q1T_THREADS, 1) k_pipe_q1_tma(const __grid_con
     if (!s_last) return;
     __threadfence();
     __shared__ Slot16 s_raw[G * 6];
-    if (threadIdx.x < G * 6) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * G * 6 + threadIdx.x].hi);
-            t += get_i128(x);
-        }
-        put_i128(&s_raw[threadIdx.x], t);
-    }
+    fold_grid_parts(parts, G * 6, s_raw, FkI128Sum());
     __syncthreads();
     // the plan's [ngroups][naggs+1] layout (slot naggs = row count = COUNT)
     for (int k = threadIdx.x; k < map.ngroups * (map.naggs + 1); k += blockDim.x) {
@@ -927,19 +946,8 @@ __global__ void __launch_bounds__(SC_THREADS) k_pipe_scalar(const __grid_constan
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x < 2) {
-        Slot16 r;
-        r.lo = __ldcg(&parts[threadIdx.x].lo);
-        r.hi = __ldcg(&parts[threadIdx.x].hi);
-        for (unsigned b = 1; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
-            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
-            else put_i128(&r, get_i128(r) + get_i128(x));
-        }
-        s_raw2[threadIdx.x] = r;
-    }
+    fold_grid_parts(parts, 2, s_raw2,
+                    [](int k) { return (k == 0 && IsFloat<VA>::value) ? (int)FK_F64_SUM : (int)FK_I128_SUM; });
     __syncthreads();
     if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
 }
@@ -1087,19 +1095,8 @@ __global__ void __launch_bounds__(SCT_THREADS, 1) k_pipe_scalar_tma(const __grid
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x < 2) {
-        Slot16 r;
-        r.lo = __ldcg(&parts[threadIdx.x].lo);
-        r.hi = __ldcg(&parts[threadIdx.x].hi);
-        for (unsigned b = 1; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
-            if (threadIdx.x == 0 && IsFloat<VA>::value) put_f64(&r, get_f64(r) + get_f64(x));
-            else put_i128(&r, get_i128(r) + get_i128(x));
-        }
-        s_raw2[threadIdx.x] = r;
-    }
+    fold_grid_parts(parts, 2, s_raw2,
+                    [](int k) { return (k == 0 && IsFloat<VA>::value) ? (int)FK_F64_SUM : (int)FK_I128_SUM; });
     __syncthreads();
     if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
 }
@@ -1405,16 +1402,7 @@ __global__ void __launch_bounds__(GF_THREADS, 1) k_pipe_gf(const __grid_constant
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    for (int k = threadIdx.x; k < NS; k += GF_THREADS) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
-            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
-            t += get_i128(x);
-        }
-        put_i128(&out[k], t);
-    }
+    fold_grid_parts(parts, NS, out, FkI128Sum());
 }
 
 // ============================================================================
@@ -1805,16 +1793,7 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x < NS) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * NS + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * NS + threadIdx.x].hi);
-            t += get_i128(x);
-        }
-        put_i128(&out[threadIdx.x], t);
-    }
+    fold_grid_parts(parts, NS, out, FkI128Sum());
 }
 
 // ============================================================================
@@ -2060,16 +2039,7 @@ __global__ void __launch_bounds__(FKG_THREADS, 1) k_pipe_fkg(const __grid_consta
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    for (int k = threadIdx.x; k < NS; k += FKG_THREADS) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
-            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
-            t += get_i128(x);
-        }
-        put_i128(&out[k], t);
-    }
+    fold_grid_parts(parts, NS, out, FkI128Sum());
 }
 
 // ---- FK grouped fold with per-thread private group slots ----------------------
@@ -2293,16 +2263,7 @@ __global__ void __launch_bounds__(FKP_THREADS, 1) k_pipe_fkg_priv(const __grid_c
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    for (int k = threadIdx.x; k < NS; k += FKP_THREADS) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * NS + k].lo);
-            x.hi = __ldcg(&parts[(size_t)b * NS + k].hi);
-            t += get_i128(x);
-        }
-        put_i128(&out[k], t);
-    }
+    fold_grid_parts(parts, NS, out, FkI128Sum());
 }
 
 // ============================================================================
@@ -2496,16 +2457,7 @@ __device__ __forceinline__ void scalar2_finish(int64_t sum, int64_t cnt, Slot16*
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x < 2) {
-        i128 t = 0;
-        for (unsigned b = 0; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
-            t += get_i128(x);
-        }
-        put_i128(&s_raw2[threadIdx.x], t);
-    }
+    fold_grid_parts(parts, 2, s_raw2, FkI128Sum());
     __syncthreads();
     if (threadIdx.x <= naggs) {
         const int src = (threadIdx.x == naggs || threadIdx.x == cnt_slot) ? 1 : 0;
@@ -3068,19 +3020,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x < 2) {
-        Slot16 r;
-        r.lo = __ldcg(&parts[threadIdx.x].lo);
-        r.hi = __ldcg(&parts[threadIdx.x].hi);
-        for (unsigned b = 1; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].lo);
-            x.hi = __ldcg(&parts[(size_t)b * 2 + threadIdx.x].hi);
-            if (threadIdx.x == 0) put_f64(&r, get_f64(r) + get_f64(x));
-            else put_i128(&r, get_i128(r) + get_i128(x));
-        }
-        s_raw2[threadIdx.x] = r;
-    }
+    fold_grid_parts(parts, 2, s_raw2, [](int k) { return k == 0 ? (int)FK_F64_SUM : (int)FK_I128_SUM; });
     __syncthreads();
     if (threadIdx.x <= map.naggs) out[threadIdx.x] = s_raw2[(threadIdx.x == map.naggs) ? 1 : map.src[threadIdx.x]];
 }
@@ -4541,21 +4481,9 @@ __global__ void __launch_bounds__(MF_THREADS) k_mat_fold(const __grid_constant__
     __syncthreads();
     if (!s_last) return;
     __threadfence();
-    if (threadIdx.x <= NA) {
-        const int a = threadIdx.x;
-        const bool fl = a < NA && P.agg[a].isf && P.agg[a].kind != VD_AGG_COUNT;
-        Slot16 r;
-        r.lo = __ldcg(&parts[a].lo);
-        r.hi = __ldcg(&parts[a].hi);
-        for (unsigned b = 1; b < gridDim.x; ++b) {
-            Slot16 x;
-            x.lo = __ldcg(&parts[(size_t)b * (NA + 1) + a].lo);
-            x.hi = __ldcg(&parts[(size_t)b * (NA + 1) + a].hi);
-            if (fl) put_f64(&r, get_f64(r) + get_f64(x));
-            else put_i128(&r, get_i128(r) + get_i128(x));
-        }
-        out[a] = r;
-    }
+    fold_grid_parts(parts, NA + 1, out, [&](int a) {
+        return (a < NA && P.agg[a].isf && P.agg[a].kind != VD_AGG_COUNT) ? (int)FK_F64_SUM : (int)FK_I128_SUM;
+    });
 }
 
 // The predicate's fast form: <= 2 interval terms on ONE 16-byte aligned

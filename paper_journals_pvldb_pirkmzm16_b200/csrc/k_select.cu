@@ -524,13 +524,13 @@ constexpr int SC_CW = 16;
 constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
 constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
-constexpr int SC_STG = 1024 + 32 + 8;        // per-warp position stage (ints, padded 1 per 32)
-constexpr int SC_PF = 4;                     // phase 2: chunks in flight per warp
-constexpr int SC_SPARSE = 64;                // phase 2: branching chunks this sparse store directly
+constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
+constexpr int SC_PF = 2;                     // phase 2: 4-chunk groups in flight per warp
+constexpr int SC_SPARSE = 128;               // phase 2: branching groups this sparse store directly
 constexpr int SC_MAXCH = 12288;              // chunks per CTA (counts kept in shared memory)
 
 template <int MODE, typename T>
-__global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
+__global__ void __maxnreg__(112) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                             int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                             uint32_t* __restrict__ bits,
                                                             int64_t* __restrict__ counts,
@@ -672,108 +672,152 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
         run += s_ccnt[i];
     }
     __syncthreads();
-    // ---- phase 2: bitmap words -> positions, chunk by chunk, no barriers ----
-    // Lane L owns word L of a chunk (rows 32L .. 32L+31): a warp popc-prefix
-    // gives every lane its output range.  Sparse chunks (branching, at most
-    // SC_SPARSE positions) store straight to global memory; denser chunks
-    // assemble in a padded shared-memory stage (index k at k + k/32: lanes
-    // 32 positions apart hit different banks) and stream out with 16-byte
-    // stores; predicated mode always uses the stage with cursor arithmetic
-    // (every row written, qualifying rows at the cursor).  Each warp keeps the
-    // words of its next SC_PF non-empty chunks in flight (a register queue):
-    // at low selectivity the pass is otherwise one L2 round trip per chunk.
+    // ---- phase 2: bitmap words -> positions, no barriers ----
+    // A warp decodes GROUPS of 4 consecutive chunks (4096 rows, contiguous
+    // in the output): lane L loads words 4L .. 4L+3 of the group with one
+    // 16-byte load (rows 128L .. 128L+127) and a warp popc-prefix gives its
+    // output range.  Branching groups with at most SC_SPARSE positions store
+    // straight to global memory; denser chunks -- and every chunk in
+    // predicated mode (cursor arithmetic: every row written, qualifying rows
+    // at the cursor) -- are assembled per 128-row block from the chunk's 32
+    // ballot words (read back as shared-memory broadcasts) in a stage and
+    // streamed out with 16-byte stores.  Each warp keeps its next SC_PF
+    // groups' words in flight; empty groups are skipped from the counts.
     if (warp == SC_CW) return;
-    int32_t* st = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
+    int32_t* sw = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
+    uint32_t* swords = reinterpret_cast<uint32_t*>(s_off + SC_MAXCH) + warp * 128;
+    const unsigned lt = lanemask_lt();
     const int64_t base = s_base;
-    int qi[SC_PF];
-    uint32_t qw[SC_PF];
+    const int ngrp = (nch + 3) >> 2;
+    auto gcount = [&](int g) {
+        int t = 0;
+#pragma unroll
+        for (int j = 0; j < 4; ++j) t += (4 * g + j < nch) ? s_ccnt[4 * g + j] : 0;
+        return t;
+    };
+    auto gload = [&](int g) {
+        if (g >= ngrp) return make_uint4(0, 0, 0, 0);
+        const int64_t w0 = (c0 + 4 * (int64_t)g) * 32 + 4 * lane;
+        if (4 * g + 4 <= nch) return __ldcs(reinterpret_cast<const uint4*>(bits + w0));
+        uint4 x = make_uint4(0, 0, 0, 0);  // the CTA's last, partial group
+        const int valid = (nch - 4 * g) * 32;  // words
+        if (4 * lane + 0 < valid) x.x = __ldcs(bits + w0 + 0);
+        if (4 * lane + 1 < valid) x.y = __ldcs(bits + w0 + 1);
+        if (4 * lane + 2 < valid) x.z = __ldcs(bits + w0 + 2);
+        if (4 * lane + 3 < valid) x.w = __ldcs(bits + w0 + 3);
+        return x;
+    };
+    int qg[SC_PF];
+    uint4 qw[SC_PF];
     int nxt = warp;
 #pragma unroll
     for (int u = 0; u < SC_PF; ++u) {
-        while (nxt < nch && s_ccnt[nxt] == 0) nxt += SC_CW;
-        qi[u] = nxt;
-        qw[u] = nxt < nch ? __ldcs(&bits[(c0 + nxt) * 32 + lane]) : 0u;
-        if (nxt < nch) nxt += SC_CW;
+        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_CW;
+        qg[u] = nxt;
+        qw[u] = gload(nxt);
+        if (nxt < ngrp) nxt += SC_CW;
     }
-    while (qi[0] < nch) {
-        const int i = qi[0];
-        const uint32_t w = qw[0];
+    while (qg[0] < ngrp) {
+        const int g = qg[0];
+        const uint4 w4 = qw[0];
 #pragma unroll
         for (int u = 0; u + 1 < SC_PF; ++u) {
-            qi[u] = qi[u + 1];
+            qg[u] = qg[u + 1];
             qw[u] = qw[u + 1];
         }
-        while (nxt < nch && s_ccnt[nxt] == 0) nxt += SC_CW;
-        qi[SC_PF - 1] = nxt;
-        qw[SC_PF - 1] = nxt < nch ? __ldcs(&bits[(c0 + nxt) * 32 + lane]) : 0u;
-        if (nxt < nch) nxt += SC_CW;
-        const int pc = __popc(w);
-        int incl = pc;
-#pragma unroll
-        for (int o = 1; o < 32; o <<= 1) {
-            const int u = __shfl_up_sync(VD_FULL, incl, o);
-            if (lane >= o) incl += u;
-        }
-        const int excl = incl - pc;
-        const int total = s_ccnt[i];
-        const int64_t g0 = base + s_off[i];
-        const int32_t row0 = (int32_t)((c0 + i) * 1024 + lane * 32);
+        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_CW;
+        qg[SC_PF - 1] = nxt;
+        qw[SC_PF - 1] = gload(nxt);
+        if (nxt < ngrp) nxt += SC_CW;
+        const int total = gcount(g);
+        const int64_t g0 = base + s_off[4 * g];
         if (MODE == 0 && total <= SC_SPARSE) {
-            uint32_t m = w;
-            int k = excl;
-            while (m) {
-                __stcs(&out[g0 + k], row0 + (__ffs(m) - 1));
-                ++k;
-                m &= m - 1;
+            const uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
+            const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
+            int incl = pc;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const int u = __shfl_up_sync(VD_FULL, incl, o);
+                if (lane >= o) incl += u;
+            }
+            int k = incl - pc;
+            const int32_t row0 = (int32_t)((c0 + 4 * (int64_t)g) * 1024 + lane * 128);
+#pragma unroll
+            for (int j = 0; j < 4; ++j) {
+                uint32_t m = ws[j];
+                while (m) {
+                    __stcs(&out[g0 + k], row0 + 32 * j + (__ffs(m) - 1));
+                    ++k;
+                    m &= m - 1;
+                }
             }
             continue;
         }
-        // output index k sits at stage index j = k + a (a = the output's
-        // misalignment in words), physically j + j/32: 16-byte output groups
-        // are 4-word stage groups that never straddle a pad
-        const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
-        if (MODE == 0) {
-            uint32_t m = w;
-            int k = excl + a;
-            while (m) {
-                st[k + (k >> 5)] = row0 + (__ffs(m) - 1);
-                ++k;
-                m &= m - 1;
-            }
-        } else {
-            int sel = excl + a, unsel = total + (lane * 32 - excl) + a;
+        // dense: per chunk, ballot-block staging from the chunk's 32 words
+        *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
+        __syncwarp();
+        int64_t gc = g0;
+        for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
+            const int cj = s_ccnt[4 * g + j];
+            if (cj == 0) continue;
+            uint32_t bw[32];
 #pragma unroll
-            for (int b = 0; b < 32; ++b) {
-                const int f = (w >> b) & 1u;
-                const int k = f ? sel : unsel;
-                st[k + (k >> 5)] = row0 + b;
-                sel += f;
-                unsel += 1 - f;
+            for (int k = 0; k < 32; k += 4) {
+                const uint4 x = *reinterpret_cast<const uint4*>(swords + 32 * j + k);  // broadcast
+                bw[k] = x.x; bw[k + 1] = x.y; bw[k + 2] = x.z; bw[k + 3] = x.w;
             }
+            const int64_t row0 = (c0 + 4 * (int64_t)g + j) * 1024;
+            const int a = (int)(((uintptr_t)(out + gc) >> 2) & 3);
+            int cur = a;
+#pragma unroll
+            for (int q = 0; q < 8; ++q) {
+                const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
+                int pre = cur;
+#pragma unroll
+                for (int jj = 0; jj < 4; ++jj) {
+                    const uint32_t w = bw[4 * q + jj];
+                    const int f = (w >> lane) & 1u;
+                    const int r = __popc(w & lt);
+                    const int32_t row = (int32_t)(row0 + (4 * q + jj) * 32 + lane);
+                    if (MODE == 0) {
+                        if (f) sw[pre + r] = row;
+                    } else {
+                        // cursor arithmetic: unconditional store; rows that do
+                        // not qualify land past the block's count, overwritten next
+                        const int sel_before = pre - cur + r;
+                        const int k = f ? pre + r : cur + cq + (jj * 32 + lane - sel_before);
+                        sw[k] = row;
+                    }
+                    pre += __popc(w);
+                }
+                cur += cq;
+            }
+            __syncwarp();
+            const int tot = cur - a;
+            const int ngr = (a + tot + 3) >> 2;
+            int32_t* ob = out + gc - a;  // 16-byte aligned
+            for (int v = lane; v < ngr; v += 32) {
+                const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
+                if (4 * v >= a && 4 * v + 4 <= a + tot) {
+                    __stcs(reinterpret_cast<int4*>(ob) + v, x);
+                } else {
+                    const int32_t xs[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+                    for (int e = 0; e < 4; ++e) {
+                        const int kk = 4 * v + e;
+                        if (kk >= a && kk < a + tot) __stcs(ob + kk, xs[e]);
+                    }
+                }
+            }
+            __syncwarp();
+            gc += cj;
         }
-        __syncwarp();
-        // flush: scalar stores up to the first 16-byte boundary of the output,
-        // one 128-bit streaming store per lane per 128 positions, scalar tail
-        const int h = min(total, (4 - a) & 3);
-        if (lane < h) __stcs(&out[g0 + lane], st[lane + a]);  // j < 32: no pad yet
-        const int nv = (total - h) >> 2;
-        int4* o4 = reinterpret_cast<int4*>(out + g0 + h);
-        for (int v = lane; v < nv; v += 32) {
-            const int j = h + a + 4 * v;  // a multiple of 4
-            const int32_t* g = st + j + (j >> 5);
-            __stcs(o4 + v, make_int4(g[0], g[1], g[2], g[3]));
-        }
-        for (int k = h + 4 * nv + lane; k < total; k += 32) {
-            const int j = k + a;
-            __stcs(&out[g0 + k], st[j + (j >> 5)]);
-        }
-        __syncwarp();
     }
 }
 
 static size_t sel_coop_smem(size_t tsize) {
     const size_t ring = (size_t)SC_STAGES * SC_CHUNKS * 1024 * tsize;
-    const size_t p2 = (size_t)SC_CW * SC_STG * 4 + (size_t)SC_MAXCH * 4;  // stages + chunk offsets
+    const size_t p2 = (size_t)SC_CW * SC_STG * 4 + (size_t)SC_MAXCH * 4 + (size_t)SC_CW * 128 * 4;  // stages, offsets, words
     return std::max(ring, p2) + 2 * SC_STAGES * 8 + (size_t)SC_MAXCH * 2;
 }
 
