@@ -520,17 +520,17 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
 // costs several microseconds of L2 round trips, far above a CTA's ~1.5 us
 // per tile.
 static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
-constexpr int SC_CW = 16;
+constexpr int SC_CW = 15;  // + the producer: 16 warps, 4 per SM sub-partition (128 registers each)
 constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
 constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
 constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
-constexpr int SC_PF = 2;                     // phase 2: 4-chunk groups in flight per warp
+constexpr int SC_PF = 4;                     // phase 2: 4-chunk groups in flight per warp
 constexpr int SC_SPARSE = 128;               // phase 2: branching groups this sparse store directly
 constexpr int SC_MAXCH = 12288;              // chunks per CTA (counts kept in shared memory)
 
 template <int MODE, typename T>
-__global__ void __maxnreg__(112) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
+__global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                             int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                             uint32_t* __restrict__ bits,
                                                             int64_t* __restrict__ counts,
