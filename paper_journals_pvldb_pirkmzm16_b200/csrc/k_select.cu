@@ -526,7 +526,8 @@ constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
 constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
 constexpr int SC_PF = 4;                     // phase 2: 4-chunk groups in flight per warp
-constexpr int SC_SPARSE = 128;               // phase 2: branching groups this sparse store directly
+constexpr int SC_SPARSE = 64;                // phase 2: branching groups this sparse store directly
+constexpr int SC_ROUND = 1024;               // phase 2: outputs per staged round (a multiple of 4)
 constexpr int SC_MAXCH = 12288;              // chunks per CTA (counts kept in shared memory)
 
 template <int MODE, typename T>
@@ -753,7 +754,60 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
             continue;
         }
-        // dense: per chunk, ballot-block staging from the chunk's 32 words
+        if (MODE == 0) {
+            // lane-owned rows, positions staged in rounds of SC_ROUND outputs
+            // (stage index k at k + k/32: lanes 32 positions apart hit
+            // different banks), each round streamed out with 16-byte stores
+            uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
+            const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
+            int incl = pc;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const int u = __shfl_up_sync(VD_FULL, incl, o);
+                if (lane >= o) incl += u;
+            }
+            int k = incl - pc;  // this lane's next output rank
+            const int32_t row0 = (int32_t)((c0 + 4 * (int64_t)g) * 1024 + lane * 128);
+            // the output's misalignment in words: output rank rb + i sits at
+            // stage index i + a (physically x + x/32); SC_ROUND % 4 == 0, so
+            // every round has the same misalignment and 16-byte groups of the
+            // output are 4-word stage groups
+            const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+            const int h0 = (4 - a) & 3;
+            for (int rb = 0; rb < total; rb += SC_ROUND) {
+                const int re = min(total, rb + SC_ROUND);
+#pragma unroll
+                for (int jj = 0; jj < 4; ++jj) {  // static indices: ws stays in registers
+                    uint32_t m = ws[jj];
+                    while (m && k < re) {
+                        const int x = k - rb + a;
+                        sw[x + (x >> 5)] = row0 + 32 * jj + (__ffs(m) - 1);
+                        ++k;
+                        m &= m - 1;
+                    }
+                    ws[jj] = m;
+                }
+                __syncwarp();
+                const int cnt = re - rb;
+                const int64_t gb = g0 + rb;
+                const int h = min(cnt, h0);
+                if (lane < h) { const int x = lane + a; __stcs(&out[gb + lane], sw[x + (x >> 5)]); }
+                const int nv = (cnt - h) >> 2;
+                int4* o4 = reinterpret_cast<int4*>(out + gb + h);
+                for (int v = lane; v < nv; v += 32) {
+                    const int x = h + a + 4 * v;  // a multiple of 4: the group never straddles a pad
+                    const int32_t* q = sw + x + (x >> 5);
+                    __stcs(o4 + v, make_int4(q[0], q[1], q[2], q[3]));
+                }
+                for (int i = h + 4 * nv + lane; i < cnt; i += 32) {
+                    const int x = i + a;
+                    __stcs(&out[gb + i], sw[x + (x >> 5)]);
+                }
+                __syncwarp();
+            }
+            continue;
+        }
+        // predicated: per chunk, ballot-block staging (cursor arithmetic)
         *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
         __syncwarp();
         int64_t gc = g0;
