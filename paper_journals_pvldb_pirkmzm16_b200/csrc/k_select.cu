@@ -754,8 +754,8 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
             continue;
         }
-        if (MODE == 0) {
-            // lane-owned rows, positions staged in rounds of SC_ROUND outputs
+        if (MODE == 0 && total <= SC_ROUND) {
+            // lane-owned rows, positions staged in one round of <= SC_ROUND outputs
             // (stage index k at k + k/32: lanes 32 positions apart hit
             // different banks), each round streamed out with 16-byte stores
             uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
@@ -807,7 +807,9 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
             continue;
         }
-        // predicated: per chunk, ballot-block staging (cursor arithmetic)
+        // dense branching groups (> SC_ROUND positions: the rank ranges of a
+        // round would belong to a quarter of the lanes) and every predicated
+        // group: per chunk, ballot-block staging
         *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
         __syncwarp();
         int64_t gc = g0;
