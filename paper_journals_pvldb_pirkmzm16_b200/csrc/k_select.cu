@@ -522,6 +522,7 @@ __global__ void __launch_bounds__(BT_THREADS, 1) k_sel_bits_tma(const T* __restr
 static size_t al256(size_t b) { return (b + 255) & ~(size_t)255; }
 constexpr int SC_CW = 15;  // + the producer: 16 warps, 4 per SM sub-partition (128 registers each)
 constexpr int SC_THREADS = SC_CW * 32 + 32;  // + producer warp
+constexpr int SC_P2W = SC_CW + 1;            // phase 2: every warp decodes
 constexpr int SC_STAGES = 3;
 constexpr int SC_CHUNKS = SC_CW;             // 1024-row chunks per tile
 constexpr int SC_STG = 1024 + 128 + 8;       // per-warp position stage (ints)
@@ -535,7 +536,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
                                                             int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                             uint32_t* __restrict__ bits,
                                                             int64_t* __restrict__ counts,
-                                                            unsigned int* __restrict__ grid_bar) {
+                                                            unsigned int* __restrict__ grid_bar, int phase1_only) {
     constexpr uint32_t TB = SC_CHUNKS * 1024 * sizeof(T);  // tile bytes
     extern __shared__ __align__(128) uint8_t smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)SC_STAGES * TB);
@@ -652,7 +653,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     }
     // exclusive scan of the chunk counts -> int32 chunk offsets within the
     // CTA (in the ring's memory, free now): thread i owns a contiguous run
-    int32_t* s_off = reinterpret_cast<int32_t*>(smem) + SC_CW * SC_STG;
+    int32_t* s_off = reinterpret_cast<int32_t*>(smem) + SC_P2W * SC_STG;
     const int per = (nch + SC_THREADS - 1) / SC_THREADS;
     const int i0 = min(nch, (int)threadIdx.x * per), i1 = min(nch, i0 + per);
     int mysum = 0;
@@ -684,7 +685,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     // ballot words (read back as shared-memory broadcasts) in a stage and
     // streamed out with 16-byte stores.  Each warp keeps its next SC_PF
     // groups' words in flight; empty groups are skipped from the counts.
-    if (warp == SC_CW) return;
+    if (phase1_only) return;  // every warp, the producer's too, decodes groups
     int32_t* sw = reinterpret_cast<int32_t*>(smem) + warp * SC_STG;  // the ring's memory, reused
     uint32_t* swords = reinterpret_cast<uint32_t*>(s_off + SC_MAXCH) + warp * 128;
     const unsigned lt = lanemask_lt();
@@ -713,10 +714,10 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
     int nxt = warp;
 #pragma unroll
     for (int u = 0; u < SC_PF; ++u) {
-        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_CW;
+        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_P2W;
         qg[u] = nxt;
         qw[u] = gload(nxt);
-        if (nxt < ngrp) nxt += SC_CW;
+        if (nxt < ngrp) nxt += SC_P2W;
     }
     while (qg[0] < ngrp) {
         const int g = qg[0];
@@ -726,10 +727,10 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             qg[u] = qg[u + 1];
             qw[u] = qw[u + 1];
         }
-        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_CW;
+        while (nxt < ngrp && gcount(nxt) == 0) nxt += SC_P2W;
         qg[SC_PF - 1] = nxt;
         qw[SC_PF - 1] = gload(nxt);
-        if (nxt < ngrp) nxt += SC_CW;
+        if (nxt < ngrp) nxt += SC_P2W;
         const int total = gcount(g);
         const int64_t g0 = base + s_off[4 * g];
         if (MODE == 0 && total <= SC_SPARSE) {
@@ -873,7 +874,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
 
 static size_t sel_coop_smem(size_t tsize) {
     const size_t ring = (size_t)SC_STAGES * SC_CHUNKS * 1024 * tsize;
-    const size_t p2 = (size_t)SC_CW * SC_STG * 4 + (size_t)SC_MAXCH * 4 + (size_t)SC_CW * 128 * 4;  // stages, offsets, words
+    const size_t p2 = (size_t)SC_P2W * SC_STG * 4 + (size_t)SC_MAXCH * 4 + (size_t)SC_P2W * 128 * 4;  // stages, offsets, words
     return std::max(ring, p2) + 2 * SC_STAGES * 8 + (size_t)SC_MAXCH * 2;
 }
 
@@ -905,8 +906,15 @@ static cudaError_t run_select_coop(const T* col, T lo, T hi, int64_t n, int32_t*
     if ((nchunks + grid - 1) / grid > SC_MAXCH) return cudaErrorNotSupported;  // caller falls back
     cudaError_t e = cudaMemsetAsync(bar, 0, 4, s);
     if (e != cudaSuccess) return e;
+    // VD_SELECT_PHASE1=1 (diagnostics only: positions are NOT written) times
+    // the stream + barrier half of the kernel
+    static const int p1 = [] {
+        const char* e = getenv("VD_SELECT_PHASE1");
+        return e && strcmp(e, "1") == 0 ? 1 : 0;
+    }();
+    int phase1_only = p1;
     void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&out_pos, (void*)&out_count,
-                    (void*)&bits, (void*)&counts, (void*)&bar};
+                    (void*)&bits, (void*)&counts, (void*)&bar, (void*)&phase1_only};
     e = cudaLaunchCooperativeKernel((const void*)kern, dim3(grid), dim3(SC_THREADS), args, sm, s);
     ++*nl;
     return e;
