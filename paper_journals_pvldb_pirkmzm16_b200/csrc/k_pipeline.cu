@@ -2920,20 +2920,26 @@ constexpr int SS_NT = SS_CW * 32;
 constexpr int SS_THREADS = SS_NT + 32;
 
 struct SelSumArgs {
-    const float* v;
+    const float* v;  // filter column
+    const float* w;  // value column (TWO), else the filter column itself
     float lo, hi;
     int64_t n;
     int32_t nstages;
 };
 
-template <int MODE>
+// TWO: Fig 15's "select sum(v2) ... where v1 between": the value
+// column is a second f32 column staged beside the filter column (both
+// tiles in one stage); a NaN (epsilon) value is skipped by the fold while
+// its row counts (A5), with EPS set when the value column may hold one.
+template <int MODE, bool TWO = false, bool EPS = false>
 __global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_constant__ SelSumArgs a,
                                                                     int64_t ntiles, Slot16* __restrict__ parts,
                                                                     unsigned int* __restrict__ done,
                                                                     Slot16* __restrict__ out, const ScalarMap map) {
     extern __shared__ __align__(128) uint8_t smem[];
     __shared__ Slot16 s_raw2[2];
-    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * SS_TILE * 4);
+    constexpr int SB = (TWO ? 2 : 1) * SS_TILE * 4;  // stage bytes
+    uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)a.nstages * SB);
     uint64_t* empty = full + a.nstages;
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     if (threadIdx.x == 0) {
@@ -2946,16 +2952,18 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_
     __syncthreads();
     double sum = 0;
     int64_t cnt = 0;
-    auto row = [&](float x) {
+    auto row2 = [&](float x, float y) {
         const bool p = x >= a.lo && x <= a.hi;  // NaN (epsilon) fails both
+        const double v = (EPS && y != y) ? 0.0 : (double)y;
         if (MODE == 1) {
-            sum += p ? (double)x : 0.0;
+            sum += p ? v : 0.0;
             cnt += p;
         } else if (p) {
-            sum += (double)x;
+            sum += v;
             cnt += 1;
         }
     };
+    auto row = [&](float x) { row2(x, x); };
     if (warp == SS_CW) {
         if (lane == 0) {
             const uint64_t pol = policy_evict_first();
@@ -2965,8 +2973,10 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_
                 const int64_t tile = blockIdx.x + it * gridDim.x;
                 if (tile >= ntiles) break;
                 if (it >= a.nstages) mbar_wait(&empty[s], ph ^ 1u);
-                mbar_expect_tx(&full[s], SS_TILE * 4);
-                tma_load_1d(smem + (size_t)s * SS_TILE * 4, a.v + tile * SS_TILE, SS_TILE * 4, &full[s], pol);
+                mbar_expect_tx(&full[s], SB);
+                tma_load_1d(smem + (size_t)s * SB, a.v + tile * SS_TILE, SS_TILE * 4, &full[s], pol);
+                if (TWO)
+                    tma_load_1d(smem + (size_t)s * SB + SS_TILE * 4, a.w + tile * SS_TILE, SS_TILE * 4, &full[s], pol);
                 if (++s == a.nstages) { s = 0; ph ^= 1u; }
             }
         }
@@ -2978,23 +2988,28 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_pipe_selsum_tma(const __grid_
             const int64_t tile = blockIdx.x + it * gridDim.x;
             if (tile >= ntiles) break;
             mbar_wait(&full[s], ph);
-            const float4* st = reinterpret_cast<const float4*>(smem + (size_t)s * SS_TILE * 4);
-            float4 x[SS_TILE / 4 / SS_NT];
+            const float4* st = reinterpret_cast<const float4*>(smem + (size_t)s * SB);
+            constexpr int K = SS_TILE / 4 / SS_NT;
+            float4 x[K], y[K];
 #pragma unroll
-            for (int k = 0; k < SS_TILE / 4 / SS_NT; ++k) x[k] = st[threadIdx.x + k * SS_NT];
+            for (int k = 0; k < K; ++k) {
+                x[k] = st[threadIdx.x + k * SS_NT];
+                y[k] = TWO ? st[SS_TILE / 4 + threadIdx.x + k * SS_NT] : x[k];
+            }
             __syncwarp();
             if (lane == 0) mbar_arrive(&empty[s]);
             if (++s == a.nstages) { s = 0; ph ^= 1u; }
 #pragma unroll
-            for (int k = 0; k < SS_TILE / 4 / SS_NT; ++k) {
-                row(x[k].x);
-                row(x[k].y);
-                row(x[k].z);
-                row(x[k].w);
+            for (int k = 0; k < K; ++k) {
+                row2(x[k].x, y[k].x);
+                row2(x[k].y, y[k].y);
+                row2(x[k].z, y[k].z);
+                row2(x[k].w, y[k].w);
             }
         }
         if (blockIdx.x == 0)
-            for (int64_t r = ntiles * SS_TILE + threadIdx.x; r < a.n; r += SS_NT) row(a.v[r]);
+            for (int64_t r = ntiles * SS_TILE + threadIdx.x; r < a.n; r += SS_NT) row2(a.v[r], TWO ? a.w[r] : a.v[r]);
+        (void)row;
     }
     __shared__ Slot16 s_w[SS_THREADS / 32][2];
     const int64_t c = warp_sum_i64(cnt);
@@ -3260,27 +3275,33 @@ static vd_status try_scalar(const vd_pipeline* p, const vd_column* cols, int nco
                           : launch_scalar<0, false, true, true, true>(sa, ws, o, m, s, nl);
             set_fragment("scalar_ldg");
         }
-    } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && va == fcol[0] && al16(cols[va].data) && use_tma &&
-               f32_interval(fcmp, fc, &sslo, &sshi)) {
+    } else if (nf == 1 && t0 == VD_F32 && tva == VD_F32 && vb < 0 && al16(cols[va].data) &&
+               al16(cols[fcol[0]].data) && use_tma && f32_interval(fcmp, fc, &sslo, &sshi)) {
+        // selective sum over f32 (Fig 15 / C1): the value column is the filter
+        // column or a second one staged beside it
+        const bool two = va != fcol[0];
         SelSumArgs ss;
-        ss.v = (const float*)cols[va].data;
+        ss.v = (const float*)cols[fcol[0]].data;
+        ss.w = (const float*)cols[va].data;
         ss.lo = sslo;
         ss.hi = sshi;
         ss.n = n;
-        ss.nstages = SS_MAXSTAGES;
+        ss.nstages = two ? 3 : SS_MAXSTAGES;
         const int grid = num_sms();
         unsigned int* dn = (unsigned int*)ws;
         Slot16* parts = (Slot16*)((char*)ws + 256);
         e = cudaMemsetAsync(dn, 0, 4, s);
         if (e == cudaSuccess) {
-            const size_t smem = (size_t)ss.nstages * SS_TILE * 4 + 2 * ss.nstages * 8;
-            if (mode) {
-                cudaFuncSetAttribute(k_pipe_selsum_tma<1>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-                k_pipe_selsum_tma<1><<<grid, SS_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
-            } else {
-                cudaFuncSetAttribute(k_pipe_selsum_tma<0>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-                k_pipe_selsum_tma<0><<<grid, SS_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);
-            }
+            const size_t smem = (size_t)ss.nstages * (two ? 2 : 1) * SS_TILE * 4 + 2 * ss.nstages * 8;
+#define SS_GO(M, T, E)                                                                                   \
+    {                                                                                                    \
+        cudaFuncSetAttribute(k_pipe_selsum_tma<M, T, E>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem); \
+        k_pipe_selsum_tma<M, T, E><<<grid, SS_THREADS, smem, s>>>(ss, n / SS_TILE, parts, dn, o, m);     \
+    }
+            if (!two) { if (mode) SS_GO(1, false, false) else SS_GO(0, false, false) }
+            else if (veps) { if (mode) SS_GO(1, true, true) else SS_GO(0, true, true) }
+            else { if (mode) SS_GO(1, true, false) else SS_GO(0, true, false) }
+#undef SS_GO
             ++*nl;
             e = cudaGetLastError();
         }

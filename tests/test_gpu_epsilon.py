@@ -3,7 +3,7 @@ selective-sum fragments, and the int64 overflow proofs at the launch shape
 that actually runs.
 
 The fused fragments that serve BASELINE.json's headline configs
-(``q1_tma``, ``q1_ldg``, ``scalar_tma``) must honour vd.h's epsilon contract
+(``q1_tma``, ``q1_ldg``, ``scalar_tma``, ``selsum_tma``) must honour vd.h's epsilon contract
 exactly like the generic fragment: a term over epsilon is false (A9), an
 epsilon group-key code gives the row no group (Partition drops it), and an
 epsilon factor makes that aggregate's value epsilon -- skipped by the SUM
@@ -186,7 +186,12 @@ def test_f32_selective_sum_of_another_column_with_nan(sel_mode):
     exp_sum, exp_cnt = v[0] + r[0], p.get("count")[0]
     dx, dy = torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda()
     plan = vd.pipeline(pred_=vd.pred([[(0, "<", t)]]), sel_mode=sel_mode, aggs=[("sum", [1]), ("count",)])
-    buf, _ = run(plan, [vd.column(dx), vd.column(dy)], n, want=("scalar_tma",))
+    buf, _ = run(plan, [vd.column(dx), vd.column(dy)], n, want=("selsum_tma",))
+    # the per-row scalar fragment (VD_SCALAR_VARIANT=ldg) agrees
+    with env(VD_SCALAR_VARIANT="ldg"):
+        lbuf, _ = run(plan, [vd.column(dx), vd.column(dy)], n, want=("scalar_ldg",))
+    lgot = vd.decode_partials(lbuf, plan, float_aggs=[True])[0]
+    assert lgot[1] == exp_cnt and abs(lgot[0] - exp_sum) <= 1e-9 * abs(exp_sum)
     got = vd.decode_partials(buf, plan, float_aggs=[True])[0]
     assert got[1] == exp_cnt and got[2] == exp_cnt
     assert abs(got[0] - exp_sum) <= 1e-9 * abs(exp_sum)
