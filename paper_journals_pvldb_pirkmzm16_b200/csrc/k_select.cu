@@ -536,7 +536,8 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
                                                             int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                             uint32_t* __restrict__ bits,
                                                             int64_t* __restrict__ counts,
-                                                            unsigned int* __restrict__ grid_bar, int phase1_only) {
+                                                            unsigned int* __restrict__ grid_bar, int phase1_only,
+                                                            int round_max) {
     constexpr uint32_t TB = SC_CHUNKS * 1024 * sizeof(T);  // tile bytes
     extern __shared__ __align__(128) uint8_t smem[];
     uint64_t* full = reinterpret_cast<uint64_t*>(smem + (size_t)SC_STAGES * TB);
@@ -755,7 +756,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
             continue;
         }
-        if (MODE == 0 && total <= SC_ROUND) {
+        if (MODE == 0 && total <= round_max) {
             // lane-owned rows, positions staged in one round of <= SC_ROUND outputs
             // (stage index k at k + k/32: lanes 32 positions apart hit
             // different banks), each round streamed out with 16-byte stores
@@ -808,10 +809,38 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             }
             continue;
         }
-        // dense branching groups (> SC_ROUND positions: the rank ranges of a
-        // round would belong to a quarter of the lanes) and every predicated
-        // group: per chunk, ballot-block staging
+        // dense groups (> SC_ROUND positions: the rank ranges of a round
+        // would belong to a quarter of the lanes) and every predicated group:
+        // per chunk, from its 32 ballot words (shared-memory broadcasts)
         *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
+        if (MODE == 0) {
+            // branching: qualifying lanes store straight to global memory --
+            // the lanes of one ballot write a run of consecutive ranks, so a
+            // store instruction covers one or two sectors, no stage round trip
+            __syncwarp();
+            int64_t gcb = g0;
+            for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
+                const int cj = s_ccnt[4 * g + j];
+                if (cj == 0) continue;
+                int32_t* ob = out + gcb;
+                const int32_t row0 = (int32_t)((c0 + 4 * (int64_t)g + j) * 1024 + lane);
+                int cur = 0;
+#pragma unroll
+                for (int k = 0; k < 32; k += 4) {
+                    const uint4 x = *reinterpret_cast<const uint4*>(swords + 32 * j + k);  // broadcast
+                    const uint32_t wk[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+                    for (int e = 0; e < 4; ++e) {
+                        const uint32_t w = wk[e];
+                        if ((w >> lane) & 1u) __stcs(ob + cur + __popc(w & lt), row0 + (k + e) * 32);
+                        cur += __popc(w);
+                    }
+                }
+                gcb += cj;
+            }
+            __syncwarp();
+            continue;
+        }
         __syncwarp();
         int64_t gc = g0;
         for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
@@ -913,8 +942,17 @@ static cudaError_t run_select_coop(const T* col, T lo, T hi, int64_t n, int32_t*
         return e && strcmp(e, "1") == 0 ? 1 : 0;
     }();
     int phase1_only = p1;
+    // branching groups with <= round_max positions take the staged lane-owned
+    // path, denser ones the direct ballot-block stores (VD_SELECT_ROUND_MAX:
+    // comparison runs; <= SC_ROUND)
+    static const int rmax = [] {
+        const char* e = getenv("VD_SELECT_ROUND_MAX");
+        const int v = e ? atoi(e) : SC_ROUND;
+        return v < 0 ? 0 : (v > SC_ROUND ? SC_ROUND : v);
+    }();
+    int round_max = rmax;
     void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&out_pos, (void*)&out_count,
-                    (void*)&bits, (void*)&counts, (void*)&bar, (void*)&phase1_only};
+                    (void*)&bits, (void*)&counts, (void*)&bar, (void*)&phase1_only, (void*)&round_max};
     e = cudaLaunchCooperativeKernel((const void*)kern, dim3(grid), dim3(SC_THREADS), args, sm, s);
     ++*nl;
     return e;
