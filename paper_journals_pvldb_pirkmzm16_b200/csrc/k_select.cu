@@ -813,34 +813,6 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
         // would belong to a quarter of the lanes) and every predicated group:
         // per chunk, from its 32 ballot words (shared-memory broadcasts)
         *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
-        if (MODE == 0) {
-            // branching: qualifying lanes store straight to global memory --
-            // the lanes of one ballot write a run of consecutive ranks, so a
-            // store instruction covers one or two sectors, no stage round trip
-            __syncwarp();
-            int64_t gcb = g0;
-            for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
-                const int cj = s_ccnt[4 * g + j];
-                if (cj == 0) continue;
-                int32_t* ob = out + gcb;
-                const int32_t row0 = (int32_t)((c0 + 4 * (int64_t)g + j) * 1024 + lane);
-                int cur = 0;
-#pragma unroll
-                for (int k = 0; k < 32; k += 4) {
-                    const uint4 x = *reinterpret_cast<const uint4*>(swords + 32 * j + k);  // broadcast
-                    const uint32_t wk[4] = {x.x, x.y, x.z, x.w};
-#pragma unroll
-                    for (int e = 0; e < 4; ++e) {
-                        const uint32_t w = wk[e];
-                        if ((w >> lane) & 1u) __stcs(ob + cur + __popc(w & lt), row0 + (k + e) * 32);
-                        cur += __popc(w);
-                    }
-                }
-                gcb += cj;
-            }
-            __syncwarp();
-            continue;
-        }
         __syncwarp();
         int64_t gc = g0;
         for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
@@ -943,8 +915,9 @@ static cudaError_t run_select_coop(const T* col, T lo, T hi, int64_t n, int32_t*
     }();
     int phase1_only = p1;
     // branching groups with <= round_max positions take the staged lane-owned
-    // path, denser ones the direct ballot-block stores (VD_SELECT_ROUND_MAX:
-    // comparison runs; <= SC_ROUND)
+    // path, denser ones the ballot-block stage (VD_SELECT_ROUND_MAX: comparison
+    // runs; <= SC_ROUND).  Storing dense groups straight from the ballot
+    // blocks (no stage) was measured slower: 1.51 vs 1.26 ms at s = 0.5.
     static const int rmax = [] {
         const char* e = getenv("VD_SELECT_ROUND_MAX");
         const int v = e ? atoi(e) : SC_ROUND;
