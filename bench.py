@@ -66,6 +66,7 @@ def parse():
     ap.add_argument("--cpu-seconds", type=float, default=10.0)
     ap.add_argument("--seed", type=int, default=0x5EEDC0DE)
     ap.add_argument("--no-graph", action="store_true", help="N > 1: launch eagerly instead of CUDA graphs")
+    ap.add_argument("--graph", action="store_true", help="replay the step as CUDA graphs at N = 1 too")
     ap.add_argument("--grouping", default="direct", choices=["direct", "hash"],
                     help="q15: identity-hashed table over min..max (vd_group_fold) or open addressing "
                          "(vd_hash_group_fold)")
@@ -489,7 +490,7 @@ def main():
     # N > 1: the two halves of the step replayed as CUDA graphs (launch
     # latency off the critical path of ~0.4 ms shards); N = 1 runs eagerly
     graphs = None
-    if world > 1 and comm.backend == "nccl" and not args.no_graph:
+    if ((world > 1 and comm.backend == "nccl") or args.graph) and not args.no_graph:
         try:
             g1, g2 = torch.cuda.CUDAGraph(), torch.cuda.CUDAGraph()
             side = torch.cuda.Stream(device=dev)

@@ -69,3 +69,15 @@ def test_nccl_two_gpus_merge_equals_one(workload):
     two = _bench(common + ["--gpus", "2"], nproc=2)
     assert two["n_gpus"] == 2 and two["cuda_graphs"] == "pipeline + (all-gather, merge)"
     assert two["result_digest"] == one["result_digest"]
+
+
+@pytest.mark.parametrize("workload", ["q1", "q19"])
+def test_graph_replay_equals_eager(workload):
+    """The step captured as CUDA graphs (pipeline; all-gather + device merge)
+    -- what N > 1 replays -- gives the eager step's result (N = 1 here, with
+    --graph forcing the capture)."""
+    common = ["--workload", workload, "--sf", "1", "--steps", "3", "--warmup", "3", "--no-cpu-baseline", "--no-e2e"]
+    eager = _bench(common)
+    graph = _bench(common + ["--graph"])
+    assert graph["cuda_graphs"] == "pipeline + (all-gather, merge)", graph["cuda_graphs"]
+    assert graph["result_digest"] == eager["result_digest"]
