@@ -698,7 +698,8 @@ def selpos_main(args, rank, world, local):
             "vs_baseline": None, "dtype": "f32", "data": "synthetic (f32 U[0,1), gen/vd_gen.h)",
             "config": bench_config(args, "selpos", 0.0, world),
             "selected": c, "achieved_selectivity": c / n,
-            "roofline": hbm_roofline(alg, "k_sel_* (bitmap + scan + positions)", ms,
+            "roofline": hbm_roofline(alg, "k_sel_coop (one cooperative launch)" if lps == 1 else
+                                     "k_sel_bits + k_scan_i32 + k_sel_total + k_sel_write", ms,
                                      ncu_traffic(f"selpos_s{args.selectivity:g}_{args.sel_mode}", world)),
             "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
