@@ -257,3 +257,36 @@ def test_fold_scan_host_validation():
     assert L.vd_fold_scan(ctypes.byref(c), None, out, None, 0, None) == vd.VD_E_WORKSPACE
     need = vd.workspace_bytes(vd.VD_OP_FOLD_SCAN, 1000)
     assert L.vd_fold_scan(ctypes.byref(c), None, out, ctypes.c_void_p(1 << 20), need, None) == vd.VD_E_CUDA
+
+
+def test_workspace_grows_with_materialising_plans():
+    """vd_workspace_bytes(VD_OP_PIPELINE): a Break plan needs n more bytes (one
+    flag per row), a Materialize plan 4 B per row + 4 B per chunk more; a bad
+    materialize value is refused (host only, no device needed)."""
+    from paper_journals_pvldb_pirkmzm16_b200 import plans, vd
+    n = 1_000_003
+    base = vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, plans.q6())
+    brk = plans.q6()
+    brk.materialize = vd.VD_MAT_BREAK
+    chk = plans.q6()
+    chk.materialize, chk.mat_chunk = vd.VD_MAT_CHUNKS, 4096
+    assert vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, brk) >= base + n
+    nch = -(-n // 4096)
+    assert vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, chk) >= base + 4 * nch * 4096 + 4 * nch
+    bad = plans.q6()
+    bad.materialize = 7
+    with pytest.raises(vd.VdError):
+        vd.workspace_bytes(vd.VD_OP_PIPELINE, n, None, bad)
+
+
+def test_hash_and_merge_group_workspace_sizes():
+    """The open-addressing tables are sized from the distinct-key bound
+    (capacity: a power of two >= 2 x max_groups); the merge table holds
+    16-byte aggregate slots."""
+    from paper_journals_pvldb_pirkmzm16_b200 import vd
+    a = vd.hash_group_fold_ws_bytes(1000, 2)
+    b = vd.hash_group_fold_ws_bytes(100_000, 2)
+    assert b > 50 * a // 2
+    assert vd.merge_groups_ws_bytes(100_000, 2) > b  # 2 words per aggregate
+    with pytest.raises(vd.VdError):
+        vd.hash_group_fold_ws_bytes(0, 2)
