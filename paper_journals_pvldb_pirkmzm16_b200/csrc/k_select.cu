@@ -592,17 +592,11 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
             uint32_t mine = 0;
             if (c < c1) {
                 if (staged) {
-                    // the chunk's values to registers first, then the stage is
-                    // released before the ballots (a held stage stalls the ring)
                     const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
-                    T v[32];
-#pragma unroll
-                    for (int k = 0; k < 32; ++k) v[k] = src[k * 32 + lane];
-                    __syncwarp();
-                    if (lane == 0) mbar_arrive(&empty[st]);
 #pragma unroll
                     for (int k = 0; k < 32; ++k) {
-                        const uint32_t b = __ballot_sync(VD_FULL, v[k] >= lo && v[k] <= hi);  // NaN / INT_MIN fail
+                        const T v = src[k * 32 + lane];
+                        const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
                         mine = lane == k ? b : mine;
                     }
                 } else {
@@ -619,7 +613,7 @@ __global__ void __launch_bounds__(SC_THREADS, 1) k_sel_coop(const T* __restrict_
                 }
             }
             __syncwarp();
-            if (lane == 0 && !(staged && c < c1)) mbar_arrive(&empty[st]);
+            if (lane == 0) mbar_arrive(&empty[st]);
             if (++st == SC_STAGES) { st = 0; ph ^= 1u; }
             if (c < c1) {
                 bits[c * 32 + lane] = mine;
