@@ -935,6 +935,421 @@ static size_t sel_coop_ws_bytes(int64_t n) {
     return 256 + al256((size_t)4096 * 8) + al256((size_t)nchunks * 32 * 4);
 }
 
+// ---- striped, warp-specialised selection: reads and writes overlapped -----------
+// k_sel_coop's decode phase starts only after the grid barrier, so HBM idles
+// on reads while positions are written and vice versa (phase 1 alone runs at
+// the read ceiling, 0.63 ms for 1e9 f32; the decode adds 0.25-0.7 ms).  Here
+// the input is cut into SS_S global STRIPES (stripe k = chunks [k N/S,
+// (k+1) N/S), each CTA owning a contiguous sub-range of every stripe), and
+// the warps of a CTA specialise:
+//   producer (1 warp)  : streams the CTA's sub-ranges, stripe after stripe,
+//                        through a TMA ring;
+//   counters (SS_CNT)  : turn chunks into ballot words (stored) and chunk
+//                        counts (shared memory, double-buffered by stripe);
+//                        at a stripe's end one publishes the CTA's count for
+//                        it and bumps the stripe's global arrival counter;
+//   decoders (SS_DEC)  : for stripe k, once every CTA has arrived, compute
+//                        the CTA's base (the totals of the earlier stripes +
+//                        the earlier CTAs' counts of stripe k), scan the chunk
+//                        counts, and expand positions (the k_sel_coop decode),
+//                        while the counters already stream stripe k+1.
+// Output order = row order: stripe by stripe, CTA by CTA within a stripe.
+// Deadlock-free under a cooperative launch (all CTAs resident): counters wait
+// only on their own decoders (stripe k+2 reuses stripe k's buffers), decoders
+// of stripe k only on every CTA's counters of stripe k.
+constexpr int SS_CNT = 4;                         // counting warps
+constexpr int SS_DEC = 11;                        // decoding warps
+constexpr int SS_THREADS = (1 + SS_CNT + SS_DEC) * 32;
+constexpr int SS_CPT = 8;                         // chunks per tile (2 per counting warp)
+constexpr int SS_STG_N = 4;                       // ring stages
+constexpr int SS_MAXKB = 2048;                    // chunks per (stripe, CTA)
+constexpr int SS_MAXS = 64;                       // stripes
+
+struct SsShared {
+    uint64_t full[SS_STG_N], empty[SS_STG_N];
+    uint64_t ready[2], freed[2];                  // stripe buffers: counted / decoded
+    int cntw[2][SS_CNT];                          // per counting warp, per stripe buffer
+    int64_t base, run;                            // decoders: this (stripe, CTA)'s base; total of earlier stripes
+    uint16_t ccnt[2][SS_MAXKB];                   // chunk counts of a stripe's sub-range
+    int32_t off[SS_MAXKB];                        // their offsets (decoders, the current stripe)
+    uint32_t words[SS_DEC][128];                  // a group's words (shared broadcasts)
+};
+
+__device__ __forceinline__ void ss_range(int64_t nchunks, int S, int k, int G, int b, int64_t* a0, int64_t* a1) {
+    const int64_t s0 = nchunks * k / S, s1 = nchunks * (k + 1) / S;
+    *a0 = s0 + (s1 - s0) * b / G;
+    *a1 = s0 + (s1 - s0) * (b + 1) / G;
+}
+
+template <int MODE, typename T>
+__global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restrict__ col, T lo, T hi, int64_t n,
+                                                              int S, int32_t* __restrict__ out,
+                                                              int64_t* __restrict__ out_count,
+                                                              uint32_t* __restrict__ bits,
+                                                              int64_t* __restrict__ counts,       // [S][G]
+                                                              unsigned int* __restrict__ arrive,  // [S]
+                                                              int round_max) {
+    constexpr uint32_t TB = SS_CPT * 1024 * sizeof(T);
+    extern __shared__ __align__(128) uint8_t smem[];
+    int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SS_STG_N * TB);  // decoders' position stages
+    SsShared& H = *reinterpret_cast<SsShared*>(stages + SS_DEC * SC_STG);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int G = gridDim.x, b = blockIdx.x;
+    const int64_t nchunks = (n + 1023) / 1024;
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < SS_STG_N; ++i) {
+            mbar_init(&H.full[i], 1);
+            mbar_init(&H.empty[i], SS_CNT);
+        }
+        for (int i = 0; i < 2; ++i) {
+            mbar_init(&H.ready[i], 1);
+            mbar_init(&H.freed[i], SS_DEC);
+        }
+        H.run = 0;
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (warp == 0) {
+        // ---- producer: the CTA's sub-range of every stripe, in order ----
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int st = 0;
+            uint32_t ph = 0;
+            int64_t it = 0;
+            for (int k = 0; k < S; ++k) {
+                int64_t a0, a1;
+                ss_range(nchunks, S, k, G, b, &a0, &a1);
+                for (int64_t c = a0; c < a1; c += SS_CPT, ++it) {
+                    if (it >= SS_STG_N) mbar_wait(&H.empty[st], ph ^ 1u);
+                    const int64_t r0 = c * 1024, r1 = min(a1, c + SS_CPT) * 1024;
+                    if (r1 <= n) {
+                        mbar_expect_tx(&H.full[st], (uint32_t)((r1 - r0) * sizeof(T)));
+                        tma_load_1d(smem + (size_t)st * TB, col + r0, (uint32_t)((r1 - r0) * sizeof(T)), &H.full[st], pol);
+                    } else {
+                        mbar_arrive(&H.full[st]);  // the column's ragged end: loaded by the counters
+                    }
+                    if (++st == SS_STG_N) { st = 0; ph ^= 1u; }
+                }
+            }
+        }
+        return;
+    }
+    if (warp <= SS_CNT) {
+        // ---- counters ----
+        const int cw = warp - 1;
+        int st = 0;
+        uint32_t ph = 0;
+        for (int k = 0; k < S; ++k) {
+            const int sb = k & 1;
+            if (k >= 2) mbar_wait(&H.freed[sb], (uint32_t)(((k - 2) >> 1) & 1));  // decoders done with stripe k-2
+            int64_t a0, a1;
+            ss_range(nchunks, S, k, G, b, &a0, &a1);
+            int mycnt = 0;
+            for (int64_t c = a0; c < a1; c += SS_CPT) {
+                mbar_wait(&H.full[st], ph);
+                const bool staged = min(a1, c + SS_CPT) * 1024 <= n;
+                for (int h = 0; h < 2; ++h) {
+                    const int64_t ch = c + 2 * cw + h;  // this warp's chunk
+                    if (ch >= a1) continue;
+                    uint32_t mine = 0;
+                    if (staged) {
+                        const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + (2 * cw + h) * 1024;
+#pragma unroll
+                        for (int q = 0; q < 32; ++q) {
+                            const T v = src[q * 32 + lane];
+                            const uint32_t bal = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
+                            mine = lane == q ? bal : mine;
+                        }
+                    } else {
+                        for (int q = 0; q < 32; ++q) {
+                            const int64_t r = ch * 1024 + q * 32 + lane;
+                            bool f = false;
+                            if (r < n) {
+                                const T v = __ldg(col + r);
+                                f = v >= lo && v <= hi;
+                            }
+                            const uint32_t bal = __ballot_sync(VD_FULL, f);
+                            mine = lane == q ? bal : mine;
+                        }
+                    }
+                    bits[ch * 32 + lane] = mine;
+                    int cc = __popc(mine);
+#pragma unroll
+                    for (int o = 16; o; o >>= 1) cc += __shfl_xor_sync(VD_FULL, cc, o);
+                    if (lane == 0) H.ccnt[sb][ch - a0] = (uint16_t)cc;
+                    mycnt += cc;
+                }
+                __syncwarp();
+                if (lane == 0) mbar_arrive(&H.empty[st]);
+                if (++st == SS_STG_N) { st = 0; ph ^= 1u; }
+            }
+            if (lane == 0) H.cntw[sb][cw] = mycnt;
+            bar_sync_n(1, SS_CNT * 32);  // every counter's words, counts of stripe k written
+            if (cw == 0 && lane == 0) {
+                int64_t t = 0;
+                for (int w = 0; w < SS_CNT; ++w) t += H.cntw[sb][w];
+                st_release_u64(reinterpret_cast<uint64_t*>(&counts[(int64_t)k * G + b]), (uint64_t)t);
+                __threadfence();
+                atomicAdd(&arrive[k], 1u);
+                mbar_arrive(&H.ready[sb]);  // release: the chunk counts and ballot words to the decoders
+            }
+        }
+        return;
+    }
+    // ---- decoders ----
+    const int dw = warp - 1 - SS_CNT;
+    const unsigned lt = lanemask_lt();
+    int32_t* sw = stages + dw * SC_STG;
+    uint32_t* swords = H.words[dw];
+    for (int k = 0; k < S; ++k) {
+        const int sb = k & 1;
+        mbar_wait(&H.ready[sb], (uint32_t)((k >> 1) & 1));
+        if (dw == 0) {
+            if (lane == 0)
+                while (ld_acquire_u32(&arrive[k]) < (unsigned)G) __nanosleep(64);
+            __syncwarp();
+            // base = earlier stripes' total + this stripe's earlier CTAs
+            int64_t before = 0, all = 0;
+            for (int i = lane; i < G; i += 32) {
+                const int64_t x = (int64_t)ld_acquire_u64(reinterpret_cast<uint64_t*>(&counts[(int64_t)k * G + i]));
+                all += x;
+                before += i < b ? x : 0;
+            }
+            before = warp_sum_i64(before);
+            all = warp_sum_i64(all);
+            if (lane == 0) {
+                H.base = H.run + before;
+                H.run += all;
+                if (k == S - 1 && b == G - 1) *out_count = H.run;
+            }
+        }
+        int64_t a0, a1;
+        ss_range(nchunks, S, k, G, b, &a0, &a1);
+        const int nch = (int)(a1 - a0);
+        // exclusive scan of the stripe's chunk counts (decoders only)
+        {
+            const int t = dw * 32 + lane, nt = SS_DEC * 32;
+            const int per = (nch + nt - 1) / nt;
+            const int i0 = min(nch, t * per), i1 = min(nch, i0 + per);
+            int my = 0;
+            for (int i = i0; i < i1; ++i) my += H.ccnt[sb][i];
+            int incl = my;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const int u = __shfl_up_sync(VD_FULL, incl, o);
+                if (lane >= o) incl += u;
+            }
+            __shared__ int s_wsum[SS_DEC];
+            if (lane == 31) s_wsum[dw] = incl;
+            bar_sync_n(2, SS_DEC * 32);
+            int wb = 0;
+            for (int w = 0; w < dw; ++w) wb += s_wsum[w];
+            int run = wb + incl - my;
+            for (int i = i0; i < i1; ++i) {
+                H.off[i] = run;
+                run += H.ccnt[sb][i];
+            }
+            bar_sync_n(2, SS_DEC * 32);
+        }
+        const int64_t base = H.base;
+        // decode 4-chunk groups of the sub-range (the k_sel_coop decode)
+        const int ngrp = (nch + 3) >> 2;
+        for (int g = dw; g < ngrp; g += SS_DEC) {
+            int total = 0;
+#pragma unroll
+            for (int j = 0; j < 4; ++j) total += (4 * g + j < nch) ? H.ccnt[sb][4 * g + j] : 0;
+            if (total == 0) continue;
+            const int64_t w0 = (a0 + 4 * (int64_t)g) * 32 + 4 * lane;
+            uint4 w4 = make_uint4(0, 0, 0, 0);
+            if (4 * g + 4 <= nch) {
+                w4 = __ldcg(reinterpret_cast<const uint4*>(bits + w0));
+            } else {
+                const int valid = (nch - 4 * g) * 32;
+                if (4 * lane + 0 < valid) w4.x = __ldcg(bits + w0 + 0);
+                if (4 * lane + 1 < valid) w4.y = __ldcg(bits + w0 + 1);
+                if (4 * lane + 2 < valid) w4.z = __ldcg(bits + w0 + 2);
+                if (4 * lane + 3 < valid) w4.w = __ldcg(bits + w0 + 3);
+            }
+            const int64_t g0 = base + H.off[4 * g];
+            if (MODE == 0 && total <= SC_SPARSE) {
+                const uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
+                const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
+                int incl = pc;
+#pragma unroll
+                for (int o = 1; o < 32; o <<= 1) {
+                    const int u = __shfl_up_sync(VD_FULL, incl, o);
+                    if (lane >= o) incl += u;
+                }
+                int kk = incl - pc;
+                const int32_t row0 = (int32_t)((a0 + 4 * (int64_t)g) * 1024 + lane * 128);
+#pragma unroll
+                for (int j = 0; j < 4; ++j) {
+                    uint32_t m = ws[j];
+                    while (m) {
+                        __stcs(&out[g0 + kk], row0 + 32 * j + (__ffs(m) - 1));
+                        ++kk;
+                        m &= m - 1;
+                    }
+                }
+                continue;
+            }
+            if (MODE == 0 && total <= round_max) {
+                uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
+                const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
+                int incl = pc;
+#pragma unroll
+                for (int o = 1; o < 32; o <<= 1) {
+                    const int u = __shfl_up_sync(VD_FULL, incl, o);
+                    if (lane >= o) incl += u;
+                }
+                int kk = incl - pc;
+                const int32_t row0 = (int32_t)((a0 + 4 * (int64_t)g) * 1024 + lane * 128);
+                const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
+                const int h0 = (4 - a) & 3;
+#pragma unroll
+                for (int jj = 0; jj < 4; ++jj) {
+                    uint32_t m = ws[jj];
+                    while (m) {
+                        const int x = kk + a;
+                        sw[x + (x >> 5)] = row0 + 32 * jj + (__ffs(m) - 1);
+                        ++kk;
+                        m &= m - 1;
+                    }
+                }
+                __syncwarp();
+                const int h = min(total, h0);
+                if (lane < h) { const int x = lane + a; __stcs(&out[g0 + lane], sw[x + (x >> 5)]); }
+                const int nv = (total - h) >> 2;
+                int4* o4 = reinterpret_cast<int4*>(out + g0 + h);
+                for (int v = lane; v < nv; v += 32) {
+                    const int x = h + a + 4 * v;
+                    const int32_t* q = sw + x + (x >> 5);
+                    __stcs(o4 + v, make_int4(q[0], q[1], q[2], q[3]));
+                }
+                for (int i = h + 4 * nv + lane; i < total; i += 32) {
+                    const int x = i + a;
+                    __stcs(&out[g0 + i], sw[x + (x >> 5)]);
+                }
+                __syncwarp();
+                continue;
+            }
+            // dense branching / predicated: per chunk, ballot-block staging
+            *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
+            __syncwarp();
+            int64_t gc = g0;
+            for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
+                const int cj = H.ccnt[sb][4 * g + j];
+                if (cj == 0) continue;
+                uint32_t bw[32];
+#pragma unroll
+                for (int q = 0; q < 32; q += 4) {
+                    const uint4 x = *reinterpret_cast<const uint4*>(swords + 32 * j + q);
+                    bw[q] = x.x; bw[q + 1] = x.y; bw[q + 2] = x.z; bw[q + 3] = x.w;
+                }
+                const int64_t row0 = (a0 + 4 * (int64_t)g + j) * 1024;
+                const int a = (int)(((uintptr_t)(out + gc) >> 2) & 3);
+                int cur = a;
+#pragma unroll
+                for (int q = 0; q < 8; ++q) {
+                    const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
+                    int pre = cur;
+#pragma unroll
+                    for (int jj = 0; jj < 4; ++jj) {
+                        const uint32_t w = bw[4 * q + jj];
+                        const int f = (w >> lane) & 1u;
+                        const int r = __popc(w & lt);
+                        const int32_t row = (int32_t)(row0 + (4 * q + jj) * 32 + lane);
+                        if (MODE == 0) {
+                            if (f) sw[pre + r] = row;
+                        } else {
+                            const int sel_before = pre - cur + r;
+                            const int kx = f ? pre + r : cur + cq + (jj * 32 + lane - sel_before);
+                            sw[kx] = row;
+                        }
+                        pre += __popc(w);
+                    }
+                    cur += cq;
+                }
+                __syncwarp();
+                const int tot = cur - a;
+                const int ngr = (a + tot + 3) >> 2;
+                int32_t* ob = out + gc - a;
+                for (int v = lane; v < ngr; v += 32) {
+                    const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
+                    if (4 * v >= a && 4 * v + 4 <= a + tot) {
+                        __stcs(reinterpret_cast<int4*>(ob) + v, x);
+                    } else {
+                        const int32_t xs[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+                        for (int e = 0; e < 4; ++e) {
+                            const int kx = 4 * v + e;
+                            if (kx >= a && kx < a + tot) __stcs(ob + kx, xs[e]);
+                        }
+                    }
+                }
+                __syncwarp();
+                gc += cj;
+            }
+        }
+        bar_sync_n(2, SS_DEC * 32);  // every decoder done with the stripe's shared state
+        if (lane == 0) mbar_arrive(&H.freed[sb]);
+    }
+}
+
+static size_t sel_stream_smem(size_t tsize) {
+    return (size_t)SS_STG_N * SS_CPT * 1024 * tsize + (size_t)SS_DEC * SC_STG * 4 + sizeof(SsShared);
+}
+
+// VD_SELECT_KERNEL=coop: the single-barrier kernel instead (comparison runs)
+static bool use_sel_stream() {
+    static const bool off = [] {
+        const char* e = getenv("VD_SELECT_KERNEL");
+        return e && strcmp(e, "coop") == 0;
+    }();
+    return !off;
+}
+
+template <int MODE, typename T>
+static cudaError_t run_select_stream(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
+                                     void* ws, cudaStream_t s, int* nl) {
+    if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
+    const int64_t nchunks = (n + 1023) / 1024;
+    const size_t sm = sel_stream_smem(sizeof(T));
+    auto kern = k_sel_stream<MODE, T>;
+    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+    int per_sm = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SS_THREADS, sm) != cudaSuccess || per_sm < 1)
+        return cudaErrorNotSupported;
+    const int G = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, 4096);
+    // stripes: enough that one stripe's decode is a small tail, few enough
+    // that every (stripe, CTA) sub-range is several tiles
+    int S = (int)std::min<int64_t>(SS_MAXS, std::max<int64_t>(1, nchunks / ((int64_t)G * 64)));
+    while (S > 1 && (nchunks / S) / G + 2 > SS_MAXKB) --S;
+    if ((nchunks / S) / G + 2 > SS_MAXKB) return cudaErrorNotSupported;  // caller falls back
+    if (nchunks < (int64_t)G * 4) return cudaErrorNotSupported;          // small inputs: the single-barrier kernel
+    char* w = (char*)ws;
+    unsigned int* arrive = (unsigned int*)w;                              // [SS_MAXS]
+    int64_t* counts = (int64_t*)(w + 256);                                // [S][G]
+    uint32_t* bits = (uint32_t*)(w + 256 + al256((size_t)SS_MAXS * 4096 * 8));
+    cudaError_t e = cudaMemsetAsync(arrive, 0, SS_MAXS * 4, s);
+    if (e != cudaSuccess) return e;
+    static const int rmax = [] {
+        const char* v = getenv("VD_SELECT_ROUND_MAX");
+        const int x = v ? atoi(v) : SC_ROUND;
+        return x < 0 ? 0 : (x > SC_ROUND ? SC_ROUND : x);
+    }();
+    int round_max = rmax;
+    void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&S, (void*)&out_pos, (void*)&out_count,
+                    (void*)&bits, (void*)&counts, (void*)&arrive, (void*)&round_max};
+    e = cudaLaunchCooperativeKernel((const void*)kern, dim3(G), dim3(SS_THREADS), args, sm, s);
+    ++*nl;
+    return e;
+}
+static size_t sel_stream_ws_bytes(int64_t n) {
+    const int64_t nchunks = (n + 1023) / 1024;
+    return 256 + al256((size_t)SS_MAXS * 4096 * 8) + al256((size_t)nchunks * 32 * 4);
+}
+
 // Per-row predicates (several columns, run heads): ballot j is word j.
 template <class F>
 __global__ void __launch_bounds__(BM_THREADS) k_sel_bits_bal(F fl, int64_t n, uint32_t* __restrict__ bits,
@@ -1114,7 +1529,7 @@ size_t select_ws_bytes(int64_t n) {
     int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
     size_t b = 256 + (size_t)ntiles * 8;
     size_t lb = (b + 255) & ~(size_t)255;
-    size_t bm = std::max(bm_ws_bytes(n), sel_coop_ws_bytes(n));
+    size_t bm = std::max(bm_ws_bytes(n), std::max(sel_coop_ws_bytes(n), sel_stream_ws_bytes(n)));
     return lb > bm ? lb : bm;
 }
 
@@ -1208,6 +1623,10 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
         if constexpr (sizeof(T) == 4) {
             if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0) {
+                if (use_sel_stream()) {
+                    cudaError_t e = run_select_stream<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+                    if (e != cudaErrorNotSupported) return e;  // else: small / too large, the single-barrier kernel
+                }
                 cudaError_t e = run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
                 if (e != cudaErrorNotSupported) return e;  // else: more chunks per CTA than fit, bitmap path
             }

@@ -82,3 +82,22 @@ def test_fused_select_i32_tiles_alternating_empty_and_full(mode):
     fn([vd.column(da)], n, vd.pred([[(0, "<", 17)]]), out_pos=out, out_count=cnt)
     k = int(cnt.item())
     assert np.array_equal(out[:k].cpu().numpy(), exp)
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("n,t", [(5 * 10**6 + 3, 0.3), (50 * 10**6 + 17, 0.02), (50 * 10**6 + 17, 0.7),
+                                 (120 * 10**6 + 1, 0.5)])
+def test_striped_select_vs_oracle(mode, n, t):
+    """The striped warp-specialised kernel (k_sel_stream: counting warps on
+    stripe k+1 while decoding warps expand stripe k, per-stripe arrival
+    counters) at sizes with 1 .. many stripes, against the oracle's
+    brute-force selection, and equal to the single-barrier kernel."""
+    v = gen.host(gen.F32_UNIFORM, n, seed=n % 1009)
+    t = float(np.float32(t))
+    pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    dv = torch.from_numpy(v).cuda()
+    got = _select(fn, dv, n, t, shift=1)
+    assert len(got) == cnt_o and np.array_equal(got, pos_o)
+    with env(VD_SELECT_KERNEL="coop"):
+        assert np.array_equal(_select(fn, dv, n, t), pos_o)
