@@ -957,10 +957,10 @@ static size_t sel_coop_ws_bytes(int64_t n) {
 // Deadlock-free under a cooperative launch (all CTAs resident): counters wait
 // only on their own decoders (stripe k+2 reuses stripe k's buffers), decoders
 // of stripe k only on every CTA's counters of stripe k.
-constexpr int SS_CNT = 4;                         // counting warps
-constexpr int SS_DEC = 11;                        // decoding warps
-constexpr int SS_THREADS = (1 + SS_CNT + SS_DEC) * 32;
-constexpr int SS_CPT = 8;                         // chunks per tile (2 per counting warp)
+constexpr int SS_WARPS = 15;                      // counting + decoding warps (CNT + DEC)
+constexpr int SS_DEC_MAX = 11;                    // decoders at the smallest CNT (4)
+constexpr int SS_THREADS = (1 + SS_WARPS) * 32;
+constexpr int SS_CPT = 8;                         // chunks per tile
 constexpr int SS_STG_N = 4;                       // ring stages
 constexpr int SS_MAXKB = 2048;                    // chunks per (stripe, CTA)
 constexpr int SS_MAXS = 64;                       // stripes
@@ -968,11 +968,11 @@ constexpr int SS_MAXS = 64;                       // stripes
 struct SsShared {
     uint64_t full[SS_STG_N], empty[SS_STG_N];
     uint64_t ready[2], freed[2];                  // stripe buffers: counted / decoded
-    int cntw[2][SS_CNT];                          // per counting warp, per stripe buffer
+    int cntw[2][SS_WARPS];                        // per counting warp, per stripe buffer
     int64_t base, run;                            // decoders: this (stripe, CTA)'s base; total of earlier stripes
     uint16_t ccnt[2][SS_MAXKB];                   // chunk counts of a stripe's sub-range
     int32_t off[SS_MAXKB];                        // their offsets (decoders, the current stripe)
-    uint32_t words[SS_DEC][128];                  // a group's words (shared broadcasts)
+    uint32_t words[SS_DEC_MAX][128];              // a group's words (shared broadcasts)
 };
 
 __device__ __forceinline__ void ss_range(int64_t nchunks, int S, int k, int G, int b, int64_t* a0, int64_t* a1) {
@@ -981,7 +981,7 @@ __device__ __forceinline__ void ss_range(int64_t nchunks, int S, int k, int G, i
     *a1 = s0 + (s1 - s0) * (b + 1) / G;
 }
 
-template <int MODE, typename T>
+template <int MODE, typename T, int CNT>
 __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                               int S, int32_t* __restrict__ out,
                                                               int64_t* __restrict__ out_count,
@@ -989,21 +989,22 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                                                               int64_t* __restrict__ counts,       // [S][G]
                                                               unsigned int* __restrict__ arrive,  // [S]
                                                               int round_max) {
+    constexpr int DEC = 15 - CNT;
     constexpr uint32_t TB = SS_CPT * 1024 * sizeof(T);
     extern __shared__ __align__(128) uint8_t smem[];
     int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SS_STG_N * TB);  // decoders' position stages
-    SsShared& H = *reinterpret_cast<SsShared*>(stages + SS_DEC * SC_STG);
+    SsShared& H = *reinterpret_cast<SsShared*>(stages + DEC * SC_STG);
     const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
     const int G = gridDim.x, b = blockIdx.x;
     const int64_t nchunks = (n + 1023) / 1024;
     if (threadIdx.x == 0) {
         for (int i = 0; i < SS_STG_N; ++i) {
             mbar_init(&H.full[i], 1);
-            mbar_init(&H.empty[i], SS_CNT);
+            mbar_init(&H.empty[i], CNT);
         }
         for (int i = 0; i < 2; ++i) {
             mbar_init(&H.ready[i], 1);
-            mbar_init(&H.freed[i], SS_DEC);
+            mbar_init(&H.freed[i], DEC);
         }
         H.run = 0;
         fence_mbar_init();
@@ -1034,7 +1035,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
         }
         return;
     }
-    if (warp <= SS_CNT) {
+    if (warp <= CNT) {
         // ---- counters ----
         const int cw = warp - 1;
         int st = 0;
@@ -1048,12 +1049,12 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
             for (int64_t c = a0; c < a1; c += SS_CPT) {
                 mbar_wait(&H.full[st], ph);
                 const bool staged = min(a1, c + SS_CPT) * 1024 <= n;
-                for (int h = 0; h < 2; ++h) {
-                    const int64_t ch = c + 2 * cw + h;  // this warp's chunk
-                    if (ch >= a1) continue;
+                for (int lc = cw; lc < SS_CPT; lc += CNT) {
+                    const int64_t ch = c + lc;  // this warp's chunk
+                    if (ch >= a1) break;
                     uint32_t mine = 0;
                     if (staged) {
-                        const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + (2 * cw + h) * 1024;
+                        const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + lc * 1024;
 #pragma unroll
                         for (int q = 0; q < 32; ++q) {
                             const T v = src[q * 32 + lane];
@@ -1084,10 +1085,10 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                 if (++st == SS_STG_N) { st = 0; ph ^= 1u; }
             }
             if (lane == 0) H.cntw[sb][cw] = mycnt;
-            bar_sync_n(1, SS_CNT * 32);  // every counter's words, counts of stripe k written
+            bar_sync_n(1, CNT * 32);  // every counter's words, counts of stripe k written
             if (cw == 0 && lane == 0) {
                 int64_t t = 0;
-                for (int w = 0; w < SS_CNT; ++w) t += H.cntw[sb][w];
+                for (int w = 0; w < CNT; ++w) t += H.cntw[sb][w];
                 st_release_u64(reinterpret_cast<uint64_t*>(&counts[(int64_t)k * G + b]), (uint64_t)t);
                 __threadfence();
                 atomicAdd(&arrive[k], 1u);
@@ -1097,7 +1098,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
         return;
     }
     // ---- decoders ----
-    const int dw = warp - 1 - SS_CNT;
+    const int dw = warp - 1 - CNT;
     const unsigned lt = lanemask_lt();
     int32_t* sw = stages + dw * SC_STG;
     uint32_t* swords = H.words[dw];
@@ -1128,7 +1129,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
         const int nch = (int)(a1 - a0);
         // exclusive scan of the stripe's chunk counts (decoders only)
         {
-            const int t = dw * 32 + lane, nt = SS_DEC * 32;
+            const int t = dw * 32 + lane, nt = DEC * 32;
             const int per = (nch + nt - 1) / nt;
             const int i0 = min(nch, t * per), i1 = min(nch, i0 + per);
             int my = 0;
@@ -1139,9 +1140,9 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                 const int u = __shfl_up_sync(VD_FULL, incl, o);
                 if (lane >= o) incl += u;
             }
-            __shared__ int s_wsum[SS_DEC];
+            __shared__ int s_wsum[DEC];
             if (lane == 31) s_wsum[dw] = incl;
-            bar_sync_n(2, SS_DEC * 32);
+            bar_sync_n(2, DEC * 32);
             int wb = 0;
             for (int w = 0; w < dw; ++w) wb += s_wsum[w];
             int run = wb + incl - my;
@@ -1149,12 +1150,12 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                 H.off[i] = run;
                 run += H.ccnt[sb][i];
             }
-            bar_sync_n(2, SS_DEC * 32);
+            bar_sync_n(2, DEC * 32);
         }
         const int64_t base = H.base;
         // decode 4-chunk groups of the sub-range (the k_sel_coop decode)
         const int ngrp = (nch + 3) >> 2;
-        for (int g = dw; g < ngrp; g += SS_DEC) {
+        for (int g = dw; g < ngrp; g += DEC) {
             int total = 0;
 #pragma unroll
             for (int j = 0; j < 4; ++j) total += (4 * g + j < nch) ? H.ccnt[sb][4 * g + j] : 0;
@@ -1291,13 +1292,13 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                 gc += cj;
             }
         }
-        bar_sync_n(2, SS_DEC * 32);  // every decoder done with the stripe's shared state
+        bar_sync_n(2, DEC * 32);  // every decoder done with the stripe's shared state
         if (lane == 0) mbar_arrive(&H.freed[sb]);
     }
 }
 
 static size_t sel_stream_smem(size_t tsize) {
-    return (size_t)SS_STG_N * SS_CPT * 1024 * tsize + (size_t)SS_DEC * SC_STG * 4 + sizeof(SsShared);
+    return (size_t)SS_STG_N * SS_CPT * 1024 * tsize + (size_t)SS_DEC_MAX * SC_STG * 4 + sizeof(SsShared);
 }
 
 // VD_SELECT_KERNEL=coop: the single-barrier kernel instead (comparison runs)
@@ -1309,13 +1310,24 @@ static bool use_sel_stream() {
     return !off;
 }
 
+// VD_SELECT_STREAM_CNT (4, 6, 8): counting warps of the 15 (tuning runs)
+static int sel_stream_cnt() {
+    static const int c = [] {
+        const char* e = getenv("VD_SELECT_STREAM_CNT");
+        const int x = e ? atoi(e) : 4;
+        return (x == 6 || x == 8) ? x : 4;
+    }();
+    return c;
+}
+
 template <int MODE, typename T>
 static cudaError_t run_select_stream(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
                                      void* ws, cudaStream_t s, int* nl) {
     if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
     const int64_t nchunks = (n + 1023) / 1024;
     const size_t sm = sel_stream_smem(sizeof(T));
-    auto kern = k_sel_stream<MODE, T>;
+    const int cnt = sel_stream_cnt();
+    auto kern = cnt == 8 ? k_sel_stream<MODE, T, 8> : cnt == 6 ? k_sel_stream<MODE, T, 6> : k_sel_stream<MODE, T, 4>;
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
     int per_sm = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SS_THREADS, sm) != cudaSuccess || per_sm < 1)
