@@ -972,7 +972,7 @@ struct SsShared {
     int64_t base, run;                            // decoders: this (stripe, CTA)'s base; total of earlier stripes
     uint16_t ccnt[2][SS_MAXKB];                   // chunk counts of a stripe's sub-range
     int32_t off[SS_MAXKB];                        // their offsets (decoders, the current stripe)
-    uint32_t words[SS_DEC_MAX][128];              // a group's words (shared broadcasts)
+    alignas(16) uint32_t words[SS_DEC_MAX][128];  // a group's words (uint4 stores)
 };
 
 __device__ __forceinline__ void ss_range(int64_t nchunks, int S, int k, int G, int b, int64_t* a0, int64_t* a1) {
