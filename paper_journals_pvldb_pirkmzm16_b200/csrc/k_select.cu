@@ -990,6 +990,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                                                               unsigned int* __restrict__ arrive,  // [S]
                                                               int round_max) {
     constexpr int DEC = 15 - CNT;
+    static_assert(sizeof(T) == 4, "k_sel_stream: 4-byte columns (f32 / i32)");
     constexpr uint32_t TB = SS_CPT * 1024 * sizeof(T);
     extern __shared__ __align__(128) uint8_t smem[];
     int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SS_STG_N * TB);  // decoders' position stages
@@ -1054,12 +1055,22 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                     if (ch >= a1) break;
                     uint32_t mine = 0;
                     if (staged) {
-                        const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + lc * 1024;
+                        // lane l builds word l (rows 32l .. 32l+31) itself from
+                        // 8 independent 16-byte loads -- no ballot chain, full
+                        // ILP for a lone warp per sub-partition; segment order
+                        // rotated by lane so a quarter-warp hits 8 distinct
+                        // bank groups (conflict-free)
+                        using V4 = typename std::conditional<IsFloat<T>::value, float4, int4>::type;
+                        const V4* src4 = reinterpret_cast<const V4*>(smem + (size_t)st * TB) + lc * 256 + lane * 8;
 #pragma unroll
-                        for (int q = 0; q < 32; ++q) {
-                            const T v = src[q * 32 + lane];
-                            const uint32_t bal = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
-                            mine = lane == q ? bal : mine;
+                        for (int i = 0; i < 8; ++i) {
+                            const int sg = (i + lane) & 7;
+                            const V4 x = src4[sg];
+                            uint32_t nib = (x.x >= lo && x.x <= hi) ? 1u : 0u;  // NaN / INT_MIN fail
+                            nib |= (x.y >= lo && x.y <= hi) ? 2u : 0u;
+                            nib |= (x.z >= lo && x.z <= hi) ? 4u : 0u;
+                            nib |= (x.w >= lo && x.w <= hi) ? 8u : 0u;
+                            mine |= nib << (4 * sg);
                         }
                     } else {
                         for (int q = 0; q < 32; ++q) {
