@@ -970,6 +970,7 @@ struct SsShared {
     uint64_t ready[2], freed[2];                  // stripe buffers: counted / decoded
     int cntw[2][SS_WARPS];                        // per counting warp, per stripe buffer
     int64_t base, run;                            // decoders: this (stripe, CTA)'s base; total of earlier stripes
+    int64_t rng[SS_MAXS + 1][2];                  // the CTA's sub-range of every stripe (no 64-bit divides in loops)
     uint16_t ccnt[2][SS_MAXKB];                   // chunk counts of a stripe's sub-range
     int32_t off[SS_MAXKB];                        // their offsets (decoders, the current stripe)
     alignas(16) uint32_t words[SS_DEC_MAX][128];  // a group's words (uint4 stores)
@@ -1010,6 +1011,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
         H.run = 0;
         fence_mbar_init();
     }
+    for (int k = threadIdx.x; k < S; k += blockDim.x) ss_range(nchunks, S, k, G, b, &H.rng[k][0], &H.rng[k][1]);
     __syncthreads();
     if (warp == 0) {
         // ---- producer: the CTA's sub-range of every stripe, in order ----
@@ -1019,8 +1021,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
             uint32_t ph = 0;
             int64_t it = 0;
             for (int k = 0; k < S; ++k) {
-                int64_t a0, a1;
-                ss_range(nchunks, S, k, G, b, &a0, &a1);
+                const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
                 for (int64_t c = a0; c < a1; c += SS_CPT, ++it) {
                     if (it >= SS_STG_N) mbar_wait(&H.empty[st], ph ^ 1u);
                     const int64_t r0 = c * 1024, r1 = min(a1, c + SS_CPT) * 1024;
@@ -1044,8 +1045,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
         for (int k = 0; k < S; ++k) {
             const int sb = k & 1;
             if (k >= 2) mbar_wait(&H.freed[sb], (uint32_t)(((k - 2) >> 1) & 1));  // decoders done with stripe k-2
-            int64_t a0, a1;
-            ss_range(nchunks, S, k, G, b, &a0, &a1);
+            const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
             int mycnt = 0;
             for (int64_t c = a0; c < a1; c += SS_CPT) {
                 mbar_wait(&H.full[st], ph);
@@ -1085,9 +1085,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                         }
                     }
                     bits[ch * 32 + lane] = mine;
-                    int cc = __popc(mine);
-#pragma unroll
-                    for (int o = 16; o; o >>= 1) cc += __shfl_xor_sync(VD_FULL, cc, o);
+                    const int cc = (int)__reduce_add_sync(VD_FULL, (unsigned)__popc(mine));  // REDUX, one instruction
                     if (lane == 0) H.ccnt[sb][ch - a0] = (uint16_t)cc;
                     mycnt += cc;
                 }
@@ -1135,8 +1133,7 @@ __global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restric
                 if (k == S - 1 && b == G - 1) *out_count = H.run;
             }
         }
-        int64_t a0, a1;
-        ss_range(nchunks, S, k, G, b, &a0, &a1);
+        const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
         const int nch = (int)(a1 - a0);
         // exclusive scan of the stripe's chunk counts (decoders only)
         {
