@@ -639,6 +639,12 @@ def main():
     comm.close()
 
 
+SEL_KERNELS = {"sel_stream": "k_sel_stream (one cooperative launch, striped)",
+               "sel_coop": "k_sel_coop (one cooperative launch, one grid barrier)",
+               "sel_bitmap": "k_sel_bits + k_scan_i32 + k_sel_total + k_sel_write",
+               "sel_lookback": "k_sel_lookback"}
+
+
 def selpos_main(args, rank, world, local):
     """C2 (Fig 1 sweep point): select v < t over 1e9 f32 -> int32 positions,
     branching or predicated (vd_select_*).  Algorithmic bytes: 4 B/row read +
@@ -674,6 +680,7 @@ def selpos_main(args, rank, world, local):
     for _ in range(max(args.warmup, 3)):
         step()
     lps = vd.last_launch_count()
+    frag = vd.last_fragment()
     torch.cuda.synchronize()
     steps = args.steps or 200
     clocks = ClockSampler(local)
@@ -698,8 +705,7 @@ def selpos_main(args, rank, world, local):
             "vs_baseline": None, "dtype": "f32", "data": "synthetic (f32 U[0,1), gen/vd_gen.h)",
             "config": bench_config(args, "selpos", 0.0, world),
             "selected": c, "achieved_selectivity": c / n,
-            "roofline": hbm_roofline(alg, "k_sel_coop (one cooperative launch)" if lps == 1 else
-                                     "k_sel_bits + k_scan_i32 + k_sel_total + k_sel_write", ms,
+            "roofline": hbm_roofline(alg, SEL_KERNELS.get(frag, frag), ms,
                                      ncu_traffic(f"selpos_s{args.selectivity:g}_{args.sel_mode}", world)),
             "clocks": clk, "e2e": None, "gpu_launches": lps * steps}
     if rank == 0 and world == 1 and not args.no_cpu_baseline:

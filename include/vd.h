@@ -547,7 +547,10 @@ int32_t vd_abi_struct_sizes(size_t* out, int32_t n);
 
 /* Name of the fragment the last vd_run_pipeline on this thread ran:
  * "q1_tma", "q1_ldg", "scalar_tma", "scalar_ldg", "selsum_tma", "gather_fold",
- * "generic", "break" or "mat_chunks" (the last two: materialising plans). */
+ * "generic", "break" or "mat_chunks" (the last two: materialising plans);
+ * after a single-term selection (vd_select_*): "sel_stream" (striped
+ * warp-specialised kernel), "sel_coop" (single grid barrier), "sel_bitmap"
+ * (bitmap + scan launches) or "sel_lookback". */
 const char* vd_last_fragment(void);
 
 /* Number of kernel launches the last successful call on this thread

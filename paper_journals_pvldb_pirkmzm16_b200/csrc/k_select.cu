@@ -961,8 +961,8 @@ constexpr int SS_WARPS = 15;                      // counting + decoding warps (
 constexpr int SS_DEC_MAX = 11;                    // decoders at the smallest CNT (4)
 constexpr int SS_THREADS = (1 + SS_WARPS) * 32;
 constexpr int SS_CPT = 8;                         // chunks per tile
-constexpr int SS_STG_N = 4;                       // ring stages
-constexpr int SS_MAXKB = 2048;                    // chunks per (stripe, CTA)
+constexpr int SS_STG_N = 5;                       // ring stages (160 KB in flight)
+constexpr int SS_MAXKB = 512;                     // chunks per (stripe, CTA)
 constexpr int SS_MAXS = 64;                       // stripes
 
 struct SsShared {
@@ -1640,17 +1640,23 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
     const int ivl = term_interval_t<T>(t, &ilo, &ihi) ? 1 : 0;
     if (aligned) {
         TermFlags<T, true> f{(const T*)p, t.cmp, t.iv, t.fv, ivl, ilo, ihi};
-        if (use_lookback()) return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+        if (use_lookback()) {
+            set_fragment("sel_lookback");
+            return run_select<MODE>(f, n, out_pos, out_count, ws, s, nl);
+        }
         if constexpr (sizeof(T) == 4) {
             if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0) {
                 if (use_sel_stream()) {
+                    set_fragment("sel_stream");
                     cudaError_t e = run_select_stream<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
                     if (e != cudaErrorNotSupported) return e;  // else: small / too large, the single-barrier kernel
                 }
+                set_fragment("sel_coop");
                 cudaError_t e = run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
                 if (e != cudaErrorNotSupported) return e;  // else: more chunks per CTA than fit, bitmap path
             }
         }
+        set_fragment("sel_bitmap");
         return run_select_bitmap<MODE>(
             [&](const BmLayout& L) {
                 bool tma_done = false;

@@ -98,6 +98,8 @@ def test_striped_select_vs_oracle(mode, n, t):
     fn = vd.select_branch if mode == "branch" else vd.select_predicated
     dv = torch.from_numpy(v).cuda()
     got = _select(fn, dv, n, t, shift=1)
+    assert vd.last_fragment() == "sel_stream"
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
     with env(VD_SELECT_KERNEL="coop"):
         assert np.array_equal(_select(fn, dv, n, t), pos_o)
+        assert vd.last_fragment() == "sel_coop"
