@@ -1310,22 +1310,17 @@ static size_t sel_stream_smem(size_t tsize) {
 }
 
 // VD_SELECT_KERNEL=coop: the single-barrier kernel instead (comparison runs)
+// (read per call: tests switch kernels inside one process)
 static bool use_sel_stream() {
-    static const bool off = [] {
-        const char* e = getenv("VD_SELECT_KERNEL");
-        return e && strcmp(e, "coop") == 0;
-    }();
-    return !off;
+    const char* e = getenv("VD_SELECT_KERNEL");
+    return !(e && strcmp(e, "coop") == 0);
 }
 
 // VD_SELECT_STREAM_CNT (4, 6, 8): counting warps of the 15 (tuning runs)
 static int sel_stream_cnt() {
-    static const int c = [] {
-        const char* e = getenv("VD_SELECT_STREAM_CNT");
-        const int x = e ? atoi(e) : 4;
-        return (x == 6 || x == 8) ? x : 4;
-    }();
-    return c;
+    const char* e = getenv("VD_SELECT_STREAM_CNT");
+    const int x = e ? atoi(e) : 4;
+    return (x == 6 || x == 8) ? x : 4;
 }
 
 template <int MODE, typename T>
