@@ -1309,12 +1309,6 @@ static size_t sel_stream_smem(size_t tsize) {
     return (size_t)SS_STG_N * SS_CPT * 1024 * tsize + (size_t)SS_DEC_MAX * SC_STG * 4 + sizeof(SsShared);
 }
 
-// VD_SELECT_KERNEL=coop: the single-barrier kernel instead (comparison runs)
-// (read per call: tests switch kernels inside one process)
-static bool use_sel_stream() {
-    const char* e = getenv("VD_SELECT_KERNEL");
-    return !(e && strcmp(e, "coop") == 0);
-}
 
 // VD_SELECT_STREAM_CNT (4, 6, 8): counting warps of the 15 (tuning runs)
 static int sel_stream_cnt() {
@@ -1540,11 +1534,397 @@ static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t*
     return cudaGetLastError();
 }
 
+// ---- lagged single-pass selection: counts published, decode SL_LAG tiles later ----
+// One cooperative persistent kernel, one CTA per SM: a producer warp streams
+// tiles t = k*G + blockIdx (SL_CW 1024-row chunks each, round robin over the
+// grid) through a TMA ring; consumer warp w, in iteration k,
+//   counts    chunk w of tile k: 32 ballots -> one row-ordered bitmap word per
+//             lane, kept in REGISTERS (a queue of SL_LAG words per lane: the
+//             predicate materialised, Fig 8's break, never written to HBM);
+//             the chunk count goes to shared memory and, once per tile, the
+//             tile's count to a global table cnt[k][blockIdx];
+//   decodes   chunk w of tile k - SL_LAG, whose output base -- the counts of
+//             every earlier tile: all of rows < k - SL_LAG of the table plus
+//             the earlier CTAs of row k - SL_LAG -- one rotating warp per
+//             iteration read from the table (SL_LAG - 1 iterations after
+//             every CTA published it, so the loads rarely wait).
+// Reads of tile k and position writes of tile k - SL_LAG overlap inside every
+// SM, with no grid barrier, no look-back chain (a base is a sum over a row
+// the CTA reads whole) and no bitmap round trip through L2: k_sel_coop's
+// decode runs only after its grid barrier (HBM idle on reads meanwhile), the
+// striped k_sel_stream splits warps between counting and decoding.
+// Deadlock-free under a cooperative launch: row j of the table is published
+// by every CTA before it waits on any row (row j - SL_LAG + 1 < j).
+constexpr int SL_CW = 15;                     // consumer warps = chunks per tile
+constexpr int SL_THREADS = (SL_CW + 1) * 32;  // + the producer warp
+constexpr int SL_STAGES = 2;                  // 2 x 60 KB in flight per SM
+constexpr int SL_NS = 8;                      // per-tile shared slots (>= SL_LAG + 2)
+constexpr int SL_LAG = 3;                     // iterations between counting and decoding a tile
+constexpr int SL_STG = 1024 + 32 + 128 + 8;   // per-warp position stage (ints): chunk + pad + garbage
+constexpr int SL_SPARSE = 48;                 // default: branching chunks this sparse store directly,
+constexpr int SL_MID = 320;                   // ... this sparse: lane-owned rows, staged (VD_SEL_SPARSE / VD_SEL_MID)
+
+struct SlShared {
+    uint64_t full[SL_STAGES], empty[SL_STAGES];
+    int cc[SL_NS][16];   // chunk counts of the tile in slot k % SL_NS
+    int off[SL_NS][16];  // their exclusive prefix within the tile
+    int64_t base[SL_NS]; // the tile's output base
+    int64_t run;         // total of the table rows read so far
+};
+
+__device__ __forceinline__ uint32_t ld_relaxed_u32(const unsigned int* p) {
+    uint32_t v;
+    asm volatile("ld.relaxed.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(p) : "memory");
+    return v;
+}
+__device__ __forceinline__ void st_relaxed_u32(unsigned int* p, uint32_t v) {
+    asm volatile("st.relaxed.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+
+// Flush stage[a, a + tot) to o[0, tot) (o - a is 16-byte aligned): 16-byte
+// streaming stores, the ragged head / tail element-wise.
+__device__ __forceinline__ void sl_flush(const int32_t* sw, int a, int tot, int32_t* o, int lane) {
+    const int ngr = (a + tot + 3) >> 2;
+    int32_t* ob = o - a;
+    for (int v = lane; v < ngr; v += 32) {
+        const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
+        if (4 * v >= a && 4 * v + 4 <= a + tot) {
+            __stcs(reinterpret_cast<int4*>(ob) + v, x);
+        } else {
+            const int32_t xs[4] = {x.x, x.y, x.z, x.w};
+#pragma unroll
+            for (int e = 0; e < 4; ++e) {
+                const int kk = 4 * v + e;
+                if (kk >= a && kk < a + tot) __stcs(ob + kk, xs[e]);
+            }
+        }
+    }
+}
+
+// Positions of one 1024-row chunk: lane L holds word L (bit i <-> row
+// row0 + 32 L + i), `cnt` its population, o = the chunk's first output.
+template <int MODE>
+__device__ __forceinline__ void sl_decode(uint32_t word, int cnt, int32_t* __restrict__ o, int32_t row0,
+                                          int32_t* __restrict__ sw, int lane, int sparse_max, int mid_max) {
+    const unsigned lt = lanemask_lt();
+    if (MODE == 1 && cnt <= mid_max) {
+        // predicated, lane-owned rows: cursor arithmetic over the lane's 32
+        // rows -- every row stored at the lane's cursor, the cursor advancing
+        // by the predicate (no branch).  A lane's writes past its last
+        // qualifying row land on the next lane's first slot; that lane
+        // re-stores its first position once all stores are done.
+        const int pc = __popc(word);
+        int incl = pc;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            const int u = __shfl_up_sync(VD_FULL, incl, d);
+            if (lane >= d) incl += u;
+        }
+        const int a = (int)(((uintptr_t)o >> 2) & 3);
+        const int k0 = incl - pc + a;
+        int cur = k0;
+        const int32_t r = row0 + 32 * lane;
+#pragma unroll
+        for (int i = 0; i < 32; ++i) {
+            sw[cur] = r + i;
+            cur += (word >> i) & 1u;
+        }
+        __syncwarp();
+        if (pc) sw[k0] = r + __ffs(word) - 1;
+        __syncwarp();
+        sl_flush(sw, a, cnt, o, lane);
+        __syncwarp();
+        return;
+    }
+    if (MODE == 0 && cnt <= mid_max) {
+        const int pc = __popc(word);
+        int incl = pc;
+#pragma unroll
+        for (int d = 1; d < 32; d <<= 1) {
+            const int u = __shfl_up_sync(VD_FULL, incl, d);
+            if (lane >= d) incl += u;
+        }
+        int k = incl - pc;
+        const int32_t r = row0 + 32 * lane - 1;
+        uint32_t m = word;
+        if (cnt <= sparse_max) {  // few positions: straight to global memory
+            while (m) {
+                __stcs(o + k, r + __ffs(m));
+                ++k;
+                m &= m - 1;
+            }
+            return;
+        }
+        // lane-owned rows staged (index x at x + x/32: lanes 32 apart hit
+        // different banks), then 16-byte stores
+        const int a = (int)(((uintptr_t)o >> 2) & 3);
+        while (m) {
+            const int x = k + a;
+            sw[x + (x >> 5)] = r + __ffs(m);
+            ++k;
+            m &= m - 1;
+        }
+        __syncwarp();
+        const int ngr = (a + cnt + 3) >> 2;
+        int32_t* ob = o - a;
+        for (int v = lane; v < ngr; v += 32) {
+            const int x = 4 * v;  // a multiple of 4: the group never straddles a pad word
+            const int32_t* q = sw + x + (x >> 5);
+            if (x >= a && x + 4 <= a + cnt) {
+                __stcs(reinterpret_cast<int4*>(ob) + v, make_int4(q[0], q[1], q[2], q[3]));
+            } else {
+#pragma unroll
+                for (int e = 0; e < 4; ++e)
+                    if (x + e >= a && x + e < a + cnt) __stcs(ob + x + e, q[e]);
+            }
+        }
+        __syncwarp();
+        return;
+    }
+    // dense chunks (and every predicated chunk): word j broadcast to the warp,
+    // lane L places row 32j + L at the running rank (branching: qualifying
+    // lanes only; predicated: cursor arithmetic -- every lane stores, rows that
+    // do not qualify past the 128-row block's count, overwritten later)
+    const int a = (int)(((uintptr_t)o >> 2) & 3);
+    int cur = a;
+    const int32_t rl = row0 + lane;
+#pragma unroll
+    for (int q = 0; q < 8; ++q) {
+        uint32_t bw[4];
+#pragma unroll
+        for (int jj = 0; jj < 4; ++jj) bw[jj] = __shfl_sync(VD_FULL, word, 4 * q + jj);
+        const int cq = __popc(bw[0]) + __popc(bw[1]) + __popc(bw[2]) + __popc(bw[3]);
+        int pre = cur;
+#pragma unroll
+        for (int jj = 0; jj < 4; ++jj) {
+            const uint32_t w = bw[jj];
+            const bool f = (w >> lane) & 1u;
+            const int r = __popc(w & lt);
+            const int32_t row = rl + 32 * (4 * q + jj);
+            if (MODE == 0) {
+                if (f) sw[pre + r] = row;
+            } else {
+                const int sel_before = pre - cur + r;
+                sw[f ? pre + r : cur + cq + (jj * 32 + lane - sel_before)] = row;
+            }
+            pre += __popc(w);
+        }
+        cur += cq;
+    }
+    __syncwarp();
+    sl_flush(sw, a, cur - a, o, lane);
+    __syncwarp();
+}
+
+template <int MODE, typename T>
+__global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__ col, T lo, T hi, int64_t n,
+                                                           int32_t* __restrict__ out, int64_t* __restrict__ out_count,
+                                                           unsigned int* __restrict__ cnt /* [nk][G], zeroed */,
+                                                           int sparse_max, int mid_max) {
+    static_assert(sizeof(T) == 4, "k_sel_lag: 4-byte columns (f32 / i32)");
+    constexpr uint32_t TB = SL_CW * 1024 * sizeof(T);
+    extern __shared__ __align__(128) uint8_t smem[];
+    int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SL_STAGES * TB);
+    SlShared& H = *reinterpret_cast<SlShared*>(stages + SL_CW * SL_STG);
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    const int G = gridDim.x, c = blockIdx.x;
+    const int64_t nchunks = (n + 1023) / 1024;
+    const int64_t ntiles = (nchunks + SL_CW - 1) / SL_CW;
+    const int64_t myk = ntiles > c ? (ntiles - c + G - 1) / G : 0;  // this CTA's tiles: k < myk
+    if (threadIdx.x == 0) {
+        for (int i = 0; i < SL_STAGES; ++i) {
+            mbar_init(&H.full[i], 1);
+            mbar_init(&H.empty[i], SL_CW);
+        }
+        H.run = 0;
+        fence_mbar_init();
+    }
+    __syncthreads();
+    if (warp == SL_CW) {  // producer
+        if (lane == 0) {
+            const uint64_t pol = policy_evict_first();
+            int st = 0;
+            uint32_t ph = 0;
+            for (int64_t k = 0; k < myk; ++k) {
+                if (k >= SL_STAGES) mbar_wait(&H.empty[st], ph ^ 1u);
+                const int64_t r0 = (k * G + c) * (int64_t)SL_CW * 1024;
+                if (r0 + (int64_t)SL_CW * 1024 <= n) {
+                    mbar_expect_tx(&H.full[st], TB);
+                    tma_load_1d(smem + (size_t)st * TB, col + r0, TB, &H.full[st], pol);
+                } else {
+                    mbar_arrive(&H.full[st]);  // the column's last, partial tile: consumers load it directly
+                }
+                if (++st == SL_STAGES) { st = 0; ph ^= 1u; }
+            }
+        }
+        return;
+    }
+    int32_t* sw = stages + warp * SL_STG;
+    uint32_t q[SL_LAG];
+#pragma unroll
+    for (int i = 0; i < SL_LAG; ++i) q[i] = 0;
+    int st = 0, rk = 0;  // rk = k % SL_CW
+    uint32_t ph = 0;
+    for (int64_t k = 0; k < myk + SL_LAG; ++k, rk = rk + 1 == SL_CW ? 0 : rk + 1) {
+        const int slot = (int)(k & (SL_NS - 1));
+        // (A) this iteration's base warp issues the loads of table row kb
+        const int64_t kb = k - SL_LAG + 1;
+        const bool role = warp == rk && kb >= 0 && kb < myk;
+        uint32_t rv[5];
+        if (role) {
+#pragma unroll
+            for (int i = 0; i < 5; ++i) {
+                const int j = lane + 32 * i;
+                rv[i] = (j < G && kb * G + j < ntiles) ? ld_relaxed_u32(cnt + kb * G + j) : 1u;  // absent tile: count 0
+            }
+        }
+        // (B) count chunk `warp` of tile k
+        uint32_t word = 0;
+        if (k < myk) {
+            mbar_wait(&H.full[st], ph);
+            const int64_t t = k * G + c;
+            const int64_t ch = t * SL_CW + warp;
+            if (ch < nchunks) {
+                if ((t + 1) * (int64_t)SL_CW * 1024 <= n) {
+                    const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
+#pragma unroll
+                    for (int j = 0; j < 32; ++j) {
+                        const T v = src[j * 32 + lane];
+                        const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
+                        word = lane == j ? b : word;
+                    }
+                } else {
+                    for (int j = 0; j < 32; ++j) {
+                        const int64_t r = ch * 1024 + j * 32 + lane;
+                        bool f = false;
+                        if (r < n) {
+                            const T v = __ldg(col + r);
+                            f = v >= lo && v <= hi;
+                        }
+                        const uint32_t b = __ballot_sync(VD_FULL, f);
+                        word = lane == j ? b : word;
+                    }
+                }
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&H.empty[st]);
+            if (++st == SL_STAGES) { st = 0; ph ^= 1u; }
+            int cw = __popc(word);
+#pragma unroll
+            for (int d = 16; d; d >>= 1) cw += __shfl_xor_sync(VD_FULL, cw, d);
+            if (lane == 0) H.cc[slot][warp] = cw;
+        }
+        // (C) base of tile kb: the earlier rows' totals + the earlier CTAs of row kb
+        if (role) {
+            int pre = 0, tot = 0;
+#pragma unroll
+            for (int i = 0; i < 5; ++i) {
+                const int j = lane + 32 * i;
+                while (rv[i] == 0u) {
+                    __nanosleep(32);
+                    rv[i] = ld_relaxed_u32(cnt + kb * G + j);
+                }
+                const int x = (int)rv[i] - 1;
+                tot += x;
+                pre += j < c ? x : 0;
+            }
+#pragma unroll
+            for (int d = 16; d; d >>= 1) {
+                pre += __shfl_xor_sync(VD_FULL, pre, d);
+                tot += __shfl_xor_sync(VD_FULL, tot, d);
+            }
+            if (lane == 0) {
+                H.base[kb & (SL_NS - 1)] = H.run + pre;
+                H.run += tot;
+            }
+        }
+        bar_sync_n(1, SL_CW * 32);
+        // (D) publish tile k: chunk offsets to shared memory, its count to the table
+        if (k < myk && warp == (rk + 7 < SL_CW ? rk + 7 : rk + 7 - SL_CW)) {
+            const int x = lane < SL_CW ? H.cc[slot][lane] : 0;
+            int incl = x;
+#pragma unroll
+            for (int d = 1; d < 32; d <<= 1) {
+                const int u = __shfl_up_sync(VD_FULL, incl, d);
+                if (lane >= d) incl += u;
+            }
+            if (lane < SL_CW) H.off[slot][lane] = incl - x;
+            if (lane == 31) st_relaxed_u32(cnt + k * G + c, (uint32_t)incl + 1u);
+        }
+        // (E) decode chunk `warp` of tile k - SL_LAG
+        const int64_t kd = k - SL_LAG;
+        if (kd >= 0) {
+            const int ds = (int)(kd & (SL_NS - 1));
+            const int cd = H.cc[ds][warp];
+            if (cd > 0) {
+                const int64_t ob = H.base[ds] + H.off[ds][warp];
+                const int32_t row0 = (int32_t)(((kd * G + c) * SL_CW + warp) * 1024);
+                sl_decode<MODE>(q[0], cd, out + ob, row0, sw, lane, sparse_max, mid_max);
+            }
+        }
+#pragma unroll
+        for (int i = 0; i + 1 < SL_LAG; ++i) q[i] = q[i + 1];
+        q[SL_LAG - 1] = word;
+    }
+    if (c == 0) {
+        bar_sync_n(1, SL_CW * 32);
+        if (threadIdx.x == 0) *out_count = H.run;
+    }
+}
+
+static size_t sel_lag_smem() {
+    return (size_t)SL_STAGES * SL_CW * 1024 * 4 + (size_t)SL_CW * SL_STG * 4 + sizeof(SlShared);
+}
+static size_t sel_lag_ws_bytes(int64_t n) {
+    const int64_t ntiles = ((n + 1023) / 1024 + SL_CW - 1) / SL_CW;
+    return al256((size_t)(ntiles + 4096) * 4);
+}
+
+// VD_SELECT_KERNEL=coop / stream: the single-barrier or striped kernel instead
+// (comparison runs; read per call: tests switch kernels inside one process)
+static int sel_kernel_choice() {
+    const char* e = getenv("VD_SELECT_KERNEL");
+    if (e && strcmp(e, "coop") == 0) return 1;
+    if (e && strcmp(e, "stream") == 0) return 2;
+    return 0;
+}
+
+template <int MODE, typename T>
+static cudaError_t run_select_lag(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
+                                  void* ws, cudaStream_t s, int* nl) {
+    if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
+    const int64_t ntiles = ((n + 1023) / 1024 + SL_CW - 1) / SL_CW;
+    const size_t sm = sel_lag_smem();
+    auto kern = k_sel_lag<MODE, T>;
+    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
+    int per_sm = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SL_THREADS, sm) != cudaSuccess || per_sm < 1)
+        return cudaErrorNotSupported;
+    const int G = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, 160);  // a table row = 5 loads per lane
+    if (ntiles < (int64_t)G * 4) return cudaErrorNotSupported;              // small inputs: the single-barrier kernel
+    if (n > (int64_t)INT32_MAX) return cudaErrorNotSupported;
+    const int64_t nk = (ntiles + G - 1) / G;
+    unsigned int* cnt = (unsigned int*)ws;
+    cudaError_t e = cudaMemsetAsync(cnt, 0, (size_t)nk * G * 4, s);
+    if (e != cudaSuccess) return e;
+    auto knob = [](const char* name, int dflt, int hi) {
+        const char* v = getenv(name);
+        const int x = v ? atoi(v) : dflt;
+        return x < 0 ? 0 : (x > hi ? hi : x);
+    };
+    int sparse_max = knob("VD_SEL_SPARSE", SL_SPARSE, 1024), mid_max = knob("VD_SEL_MID", SL_MID, 1024);
+    void* args[] = {(void*)&col,       (void*)&lo,  (void*)&hi,         (void*)&n,      (void*)&out_pos,
+                    (void*)&out_count, (void*)&cnt, (void*)&sparse_max, (void*)&mid_max};
+    e = cudaLaunchCooperativeKernel((const void*)kern, dim3(G), dim3(SL_THREADS), args, sm, s);
+    ++*nl;
+    return e;
+}
+
 size_t select_ws_bytes(int64_t n) {
     int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
     size_t b = 256 + (size_t)ntiles * 8;
     size_t lb = (b + 255) & ~(size_t)255;
-    size_t bm = std::max(bm_ws_bytes(n), std::max(sel_coop_ws_bytes(n), sel_stream_ws_bytes(n)));
+    size_t bm = std::max(std::max(bm_ws_bytes(n), sel_lag_ws_bytes(n)), std::max(sel_coop_ws_bytes(n), sel_stream_ws_bytes(n)));
     return lb > bm ? lb : bm;
 }
 
@@ -1641,7 +2021,12 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
         }
         if constexpr (sizeof(T) == 4) {
             if (ivl && use_sel_coop() && ((uintptr_t)p & 15) == 0) {
-                if (use_sel_stream()) {
+                const int kc = sel_kernel_choice();
+                if (kc == 0) {
+                    set_fragment("sel_lag");
+                    cudaError_t e = run_select_lag<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
+                    if (e != cudaErrorNotSupported) return e;  // else: small, the single-barrier kernel
+                } else if (kc == 2) {
                     set_fragment("sel_stream");
                     cudaError_t e = run_select_stream<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
                     if (e != cudaErrorNotSupported) return e;  // else: small / too large, the single-barrier kernel

@@ -86,20 +86,49 @@ def test_fused_select_i32_tiles_alternating_empty_and_full(mode):
 
 @pytest.mark.parametrize("mode", ["branch", "predicated"])
 @pytest.mark.parametrize("n,t", [(5 * 10**6 + 3, 0.3), (50 * 10**6 + 17, 0.02), (50 * 10**6 + 17, 0.7),
-                                 (120 * 10**6 + 1, 0.5)])
-def test_striped_select_vs_oracle(mode, n, t):
-    """The striped warp-specialised kernel (k_sel_stream: counting warps on
-    stripe k+1 while decoding warps expand stripe k, per-stripe arrival
-    counters) at sizes with 1 .. many stripes, against the oracle's
-    brute-force selection, and equal to the single-barrier kernel."""
+                                 (120 * 10**6 + 1, 0.5), (37 * 10**6 + 4093, 0.002), (41 * 10**6 + 9, 0.12)])
+def test_large_select_kernels_vs_oracle(mode, n, t):
+    """The large-input kernels against the oracle's brute-force selection:
+    the default lagged single pass (k_sel_lag: tile counts published to a
+    table, each tile decoded SL_LAG iterations later from register-held
+    words; sparse / lane-owned / dense chunk paths), the striped
+    warp-specialised kernel (k_sel_stream) and the single-barrier kernel
+    (k_sel_coop), at sizes with a ragged last tile, into an unaligned
+    output."""
     v = gen.host(gen.F32_UNIFORM, n, seed=n % 1009)
     t = float(np.float32(t))
     pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
     fn = vd.select_branch if mode == "branch" else vd.select_predicated
     dv = torch.from_numpy(v).cuda()
     got = _select(fn, dv, n, t, shift=1)
-    assert vd.last_fragment() == "sel_stream"
+    assert vd.last_fragment() == "sel_lag"
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
-    with env(VD_SELECT_KERNEL="coop"):
-        assert np.array_equal(_select(fn, dv, n, t), pos_o)
-        assert vd.last_fragment() == "sel_coop"
+    for kern in ("stream", "coop"):
+        with env(VD_SELECT_KERNEL=kern):
+            assert np.array_equal(_select(fn, dv, n, t), pos_o)
+            assert vd.last_fragment() == "sel_" + kern
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+def test_lag_select_chunk_density_mix(mode):
+    """Chunks of every density class of k_sel_lag's decode in one input
+    (empty, <= SL_SPARSE, <= SL_MID, dense, full) with NaN epsilon rows,
+    i32 and f32, against the oracle."""
+    n = 148 * 15 * 1024 * 6 + 12345
+    rng = np.random.default_rng(7)
+    chunk = np.arange(n) // 1024
+    dens = np.array([0.0, 0.01, 0.04, 0.2, 0.31, 0.6, 1.0])[chunk % 7]
+    v = np.where(rng.random(n) < dens, np.float32(0.25), np.float32(0.75)).astype(np.float32)
+    v[::977] = np.nan
+    pos_o, cnt_o, _ = oracle.select_f32(v, 0.5, "lt")
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    got = _select(fn, torch.from_numpy(v).cuda(), n, 0.5, shift=3)
+    assert vd.last_fragment() == "sel_lag"
+    assert len(got) == cnt_o and np.array_equal(got, pos_o)
+    a = np.where(np.isnan(v), -2**31, np.where(v < 0.5, 1, 9)).astype(np.int32)
+    out = torch.empty(n, dtype=torch.int32, device="cuda")
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    fn([vd.column(torch.from_numpy(a).cuda())], n, vd.pred([[(0, "<", 5)]]), out_pos=out, out_count=cnt)
+    assert vd.last_fragment() == "sel_lag"
+    k = int(cnt.item())
+    assert k == cnt_o and np.array_equal(out[:k].cpu().numpy(), pos_o)
