@@ -640,7 +640,6 @@ def main():
 
 
 SEL_KERNELS = {"sel_lag": "k_sel_lag (one cooperative launch, lagged decode)",
-               "sel_stream": "k_sel_stream (one cooperative launch, striped)",
                "sel_coop": "k_sel_coop (one cooperative launch, one grid barrier)",
                "sel_bitmap": "k_sel_bits + k_scan_i32 + k_sel_total + k_sel_write",
                "sel_lookback": "k_sel_lookback"}

@@ -935,429 +935,6 @@ static size_t sel_coop_ws_bytes(int64_t n) {
     return 256 + al256((size_t)4096 * 8) + al256((size_t)nchunks * 32 * 4);
 }
 
-// ---- striped, warp-specialised selection: reads and writes overlapped -----------
-// k_sel_coop's decode phase starts only after the grid barrier, so HBM idles
-// on reads while positions are written and vice versa (phase 1 alone runs at
-// the read ceiling, 0.63 ms for 1e9 f32; the decode adds 0.25-0.7 ms).  Here
-// the input is cut into SS_S global STRIPES (stripe k = chunks [k N/S,
-// (k+1) N/S), each CTA owning a contiguous sub-range of every stripe), and
-// the warps of a CTA specialise:
-//   producer (1 warp)  : streams the CTA's sub-ranges, stripe after stripe,
-//                        through a TMA ring;
-//   counters (SS_CNT)  : turn chunks into ballot words (stored) and chunk
-//                        counts (shared memory, double-buffered by stripe);
-//                        at a stripe's end one publishes the CTA's count for
-//                        it and bumps the stripe's global arrival counter;
-//   decoders (SS_DEC)  : for stripe k, once every CTA has arrived, compute
-//                        the CTA's base (the totals of the earlier stripes +
-//                        the earlier CTAs' counts of stripe k), scan the chunk
-//                        counts, and expand positions (the k_sel_coop decode),
-//                        while the counters already stream stripe k+1.
-// Output order = row order: stripe by stripe, CTA by CTA within a stripe.
-// Deadlock-free under a cooperative launch (all CTAs resident): counters wait
-// only on their own decoders (stripe k+2 reuses stripe k's buffers), decoders
-// of stripe k only on every CTA's counters of stripe k.
-constexpr int SS_WARPS = 15;                      // counting + decoding warps (CNT + DEC)
-constexpr int SS_DEC_MAX = 11;                    // decoders at the smallest CNT (4)
-constexpr int SS_THREADS = (1 + SS_WARPS) * 32;
-constexpr int SS_CPT = 8;                         // chunks per tile
-constexpr int SS_STG_N = 5;                       // ring stages (160 KB in flight)
-constexpr int SS_MAXKB = 512;                     // chunks per (stripe, CTA)
-constexpr int SS_MAXS = 64;                       // stripes
-
-struct SsShared {
-    uint64_t full[SS_STG_N], empty[SS_STG_N];
-    uint64_t ready[2], freed[2];                  // stripe buffers: counted / decoded
-    int cntw[2][SS_WARPS];                        // per counting warp, per stripe buffer
-    int64_t base, run;                            // decoders: this (stripe, CTA)'s base; total of earlier stripes
-    int64_t rng[SS_MAXS + 1][2];                  // the CTA's sub-range of every stripe (no 64-bit divides in loops)
-    uint16_t ccnt[2][SS_MAXKB];                   // chunk counts of a stripe's sub-range
-    int32_t off[SS_MAXKB];                        // their offsets (decoders, the current stripe)
-    alignas(16) uint32_t words[SS_DEC_MAX][128];  // a group's words (uint4 stores)
-};
-
-__device__ __forceinline__ void ss_range(int64_t nchunks, int S, int k, int G, int b, int64_t* a0, int64_t* a1) {
-    const int64_t s0 = nchunks * k / S, s1 = nchunks * (k + 1) / S;
-    *a0 = s0 + (s1 - s0) * b / G;
-    *a1 = s0 + (s1 - s0) * (b + 1) / G;
-}
-
-template <int MODE, typename T, int CNT>
-__global__ void __launch_bounds__(SS_THREADS, 1) k_sel_stream(const T* __restrict__ col, T lo, T hi, int64_t n,
-                                                              int S, int32_t* __restrict__ out,
-                                                              int64_t* __restrict__ out_count,
-                                                              uint32_t* __restrict__ bits,
-                                                              int64_t* __restrict__ counts,       // [S][G]
-                                                              unsigned int* __restrict__ arrive,  // [S]
-                                                              int round_max) {
-    constexpr int DEC = 15 - CNT;
-    static_assert(sizeof(T) == 4, "k_sel_stream: 4-byte columns (f32 / i32)");
-    constexpr uint32_t TB = SS_CPT * 1024 * sizeof(T);
-    extern __shared__ __align__(128) uint8_t smem[];
-    int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SS_STG_N * TB);  // decoders' position stages
-    SsShared& H = *reinterpret_cast<SsShared*>(stages + DEC * SC_STG);
-    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
-    const int G = gridDim.x, b = blockIdx.x;
-    const int64_t nchunks = (n + 1023) / 1024;
-    if (threadIdx.x == 0) {
-        for (int i = 0; i < SS_STG_N; ++i) {
-            mbar_init(&H.full[i], 1);
-            mbar_init(&H.empty[i], CNT);
-        }
-        for (int i = 0; i < 2; ++i) {
-            mbar_init(&H.ready[i], 1);
-            mbar_init(&H.freed[i], DEC);
-        }
-        H.run = 0;
-        fence_mbar_init();
-    }
-    for (int k = threadIdx.x; k < S; k += blockDim.x) ss_range(nchunks, S, k, G, b, &H.rng[k][0], &H.rng[k][1]);
-    __syncthreads();
-    if (warp == 0) {
-        // ---- producer: the CTA's sub-range of every stripe, in order ----
-        if (lane == 0) {
-            const uint64_t pol = policy_evict_first();
-            int st = 0;
-            uint32_t ph = 0;
-            int64_t it = 0;
-            for (int k = 0; k < S; ++k) {
-                const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
-                for (int64_t c = a0; c < a1; c += SS_CPT, ++it) {
-                    if (it >= SS_STG_N) mbar_wait(&H.empty[st], ph ^ 1u);
-                    const int64_t r0 = c * 1024, r1 = min(a1, c + SS_CPT) * 1024;
-                    if (r1 <= n) {
-                        mbar_expect_tx(&H.full[st], (uint32_t)((r1 - r0) * sizeof(T)));
-                        tma_load_1d(smem + (size_t)st * TB, col + r0, (uint32_t)((r1 - r0) * sizeof(T)), &H.full[st], pol);
-                    } else {
-                        mbar_arrive(&H.full[st]);  // the column's ragged end: loaded by the counters
-                    }
-                    if (++st == SS_STG_N) { st = 0; ph ^= 1u; }
-                }
-            }
-        }
-        return;
-    }
-    if (warp <= CNT) {
-        // ---- counters ----
-        const int cw = warp - 1;
-        int st = 0;
-        uint32_t ph = 0;
-        for (int k = 0; k < S; ++k) {
-            const int sb = k & 1;
-            if (k >= 2) mbar_wait(&H.freed[sb], (uint32_t)(((k - 2) >> 1) & 1));  // decoders done with stripe k-2
-            const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
-            int mycnt = 0;
-            for (int64_t c = a0; c < a1; c += SS_CPT) {
-                mbar_wait(&H.full[st], ph);
-                const bool staged = min(a1, c + SS_CPT) * 1024 <= n;
-                for (int lc = cw; lc < SS_CPT; lc += CNT) {
-                    const int64_t ch = c + lc;  // this warp's chunk
-                    if (ch >= a1) break;
-                    uint32_t mine = 0;
-                    if (staged) {
-                        // lane l builds word l (rows 32l .. 32l+31) itself from
-                        // 8 independent 16-byte loads -- no ballot chain, full
-                        // ILP for a lone warp per sub-partition; segment order
-                        // rotated by lane so a quarter-warp hits 8 distinct
-                        // bank groups (conflict-free)
-                        using V4 = typename std::conditional<IsFloat<T>::value, float4, int4>::type;
-                        const V4* src4 = reinterpret_cast<const V4*>(smem + (size_t)st * TB) + lc * 256 + lane * 8;
-#pragma unroll
-                        for (int i = 0; i < 8; ++i) {
-                            const int sg = (i + lane) & 7;
-                            const V4 x = src4[sg];
-                            uint32_t nib = (x.x >= lo && x.x <= hi) ? 1u : 0u;  // NaN / INT_MIN fail
-                            nib |= (x.y >= lo && x.y <= hi) ? 2u : 0u;
-                            nib |= (x.z >= lo && x.z <= hi) ? 4u : 0u;
-                            nib |= (x.w >= lo && x.w <= hi) ? 8u : 0u;
-                            mine |= nib << (4 * sg);
-                        }
-                    } else {
-                        for (int q = 0; q < 32; ++q) {
-                            const int64_t r = ch * 1024 + q * 32 + lane;
-                            bool f = false;
-                            if (r < n) {
-                                const T v = __ldg(col + r);
-                                f = v >= lo && v <= hi;
-                            }
-                            const uint32_t bal = __ballot_sync(VD_FULL, f);
-                            mine = lane == q ? bal : mine;
-                        }
-                    }
-                    bits[ch * 32 + lane] = mine;
-                    const int cc = (int)__reduce_add_sync(VD_FULL, (unsigned)__popc(mine));  // REDUX, one instruction
-                    if (lane == 0) H.ccnt[sb][ch - a0] = (uint16_t)cc;
-                    mycnt += cc;
-                }
-                __syncwarp();
-                if (lane == 0) mbar_arrive(&H.empty[st]);
-                if (++st == SS_STG_N) { st = 0; ph ^= 1u; }
-            }
-            if (lane == 0) H.cntw[sb][cw] = mycnt;
-            bar_sync_n(1, CNT * 32);  // every counter's words, counts of stripe k written
-            if (cw == 0 && lane == 0) {
-                int64_t t = 0;
-                for (int w = 0; w < CNT; ++w) t += H.cntw[sb][w];
-                st_release_u64(reinterpret_cast<uint64_t*>(&counts[(int64_t)k * G + b]), (uint64_t)t);
-                __threadfence();
-                atomicAdd(&arrive[k], 1u);
-                mbar_arrive(&H.ready[sb]);  // release: the chunk counts and ballot words to the decoders
-            }
-        }
-        return;
-    }
-    // ---- decoders ----
-    const int dw = warp - 1 - CNT;
-    const unsigned lt = lanemask_lt();
-    int32_t* sw = stages + dw * SC_STG;
-    uint32_t* swords = H.words[dw];
-    for (int k = 0; k < S; ++k) {
-        const int sb = k & 1;
-        mbar_wait(&H.ready[sb], (uint32_t)((k >> 1) & 1));
-        if (dw == 0) {
-            if (lane == 0)
-                while (ld_acquire_u32(&arrive[k]) < (unsigned)G) __nanosleep(64);
-            __syncwarp();
-            // base = earlier stripes' total + this stripe's earlier CTAs
-            int64_t before = 0, all = 0;
-            for (int i = lane; i < G; i += 32) {
-                const int64_t x = (int64_t)ld_acquire_u64(reinterpret_cast<uint64_t*>(&counts[(int64_t)k * G + i]));
-                all += x;
-                before += i < b ? x : 0;
-            }
-            before = warp_sum_i64(before);
-            all = warp_sum_i64(all);
-            if (lane == 0) {
-                H.base = H.run + before;
-                H.run += all;
-                if (k == S - 1 && b == G - 1) *out_count = H.run;
-            }
-        }
-        const int64_t a0 = H.rng[k][0], a1 = H.rng[k][1];
-        const int nch = (int)(a1 - a0);
-        // exclusive scan of the stripe's chunk counts (decoders only)
-        {
-            const int t = dw * 32 + lane, nt = DEC * 32;
-            const int per = (nch + nt - 1) / nt;
-            const int i0 = min(nch, t * per), i1 = min(nch, i0 + per);
-            int my = 0;
-            for (int i = i0; i < i1; ++i) my += H.ccnt[sb][i];
-            int incl = my;
-#pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                const int u = __shfl_up_sync(VD_FULL, incl, o);
-                if (lane >= o) incl += u;
-            }
-            __shared__ int s_wsum[DEC];
-            if (lane == 31) s_wsum[dw] = incl;
-            bar_sync_n(2, DEC * 32);
-            int wb = 0;
-            for (int w = 0; w < dw; ++w) wb += s_wsum[w];
-            int run = wb + incl - my;
-            for (int i = i0; i < i1; ++i) {
-                H.off[i] = run;
-                run += H.ccnt[sb][i];
-            }
-            bar_sync_n(2, DEC * 32);
-        }
-        const int64_t base = H.base;
-        // decode 4-chunk groups of the sub-range (the k_sel_coop decode)
-        const int ngrp = (nch + 3) >> 2;
-        for (int g = dw; g < ngrp; g += DEC) {
-            int total = 0;
-#pragma unroll
-            for (int j = 0; j < 4; ++j) total += (4 * g + j < nch) ? H.ccnt[sb][4 * g + j] : 0;
-            if (total == 0) continue;
-            const int64_t w0 = (a0 + 4 * (int64_t)g) * 32 + 4 * lane;
-            uint4 w4 = make_uint4(0, 0, 0, 0);
-            if (4 * g + 4 <= nch) {
-                w4 = __ldcg(reinterpret_cast<const uint4*>(bits + w0));
-            } else {
-                const int valid = (nch - 4 * g) * 32;
-                if (4 * lane + 0 < valid) w4.x = __ldcg(bits + w0 + 0);
-                if (4 * lane + 1 < valid) w4.y = __ldcg(bits + w0 + 1);
-                if (4 * lane + 2 < valid) w4.z = __ldcg(bits + w0 + 2);
-                if (4 * lane + 3 < valid) w4.w = __ldcg(bits + w0 + 3);
-            }
-            const int64_t g0 = base + H.off[4 * g];
-            if (MODE == 0 && total <= SC_SPARSE) {
-                const uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
-                const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
-                int incl = pc;
-#pragma unroll
-                for (int o = 1; o < 32; o <<= 1) {
-                    const int u = __shfl_up_sync(VD_FULL, incl, o);
-                    if (lane >= o) incl += u;
-                }
-                int kk = incl - pc;
-                const int32_t row0 = (int32_t)((a0 + 4 * (int64_t)g) * 1024 + lane * 128);
-#pragma unroll
-                for (int j = 0; j < 4; ++j) {
-                    uint32_t m = ws[j];
-                    while (m) {
-                        __stcs(&out[g0 + kk], row0 + 32 * j + (__ffs(m) - 1));
-                        ++kk;
-                        m &= m - 1;
-                    }
-                }
-                continue;
-            }
-            if (MODE == 0 && total <= round_max) {
-                uint32_t ws[4] = {w4.x, w4.y, w4.z, w4.w};
-                const int pc = __popc(ws[0]) + __popc(ws[1]) + __popc(ws[2]) + __popc(ws[3]);
-                int incl = pc;
-#pragma unroll
-                for (int o = 1; o < 32; o <<= 1) {
-                    const int u = __shfl_up_sync(VD_FULL, incl, o);
-                    if (lane >= o) incl += u;
-                }
-                int kk = incl - pc;
-                const int32_t row0 = (int32_t)((a0 + 4 * (int64_t)g) * 1024 + lane * 128);
-                const int a = (int)(((uintptr_t)(out + g0) >> 2) & 3);
-                const int h0 = (4 - a) & 3;
-#pragma unroll
-                for (int jj = 0; jj < 4; ++jj) {
-                    uint32_t m = ws[jj];
-                    while (m) {
-                        const int x = kk + a;
-                        sw[x + (x >> 5)] = row0 + 32 * jj + (__ffs(m) - 1);
-                        ++kk;
-                        m &= m - 1;
-                    }
-                }
-                __syncwarp();
-                const int h = min(total, h0);
-                if (lane < h) { const int x = lane + a; __stcs(&out[g0 + lane], sw[x + (x >> 5)]); }
-                const int nv = (total - h) >> 2;
-                int4* o4 = reinterpret_cast<int4*>(out + g0 + h);
-                for (int v = lane; v < nv; v += 32) {
-                    const int x = h + a + 4 * v;
-                    const int32_t* q = sw + x + (x >> 5);
-                    __stcs(o4 + v, make_int4(q[0], q[1], q[2], q[3]));
-                }
-                for (int i = h + 4 * nv + lane; i < total; i += 32) {
-                    const int x = i + a;
-                    __stcs(&out[g0 + i], sw[x + (x >> 5)]);
-                }
-                __syncwarp();
-                continue;
-            }
-            // dense branching / predicated: per chunk, ballot-block staging
-            *reinterpret_cast<uint4*>(swords + 4 * lane) = w4;
-            __syncwarp();
-            int64_t gc = g0;
-            for (int j = 0; j < 4 && 4 * g + j < nch; ++j) {
-                const int cj = H.ccnt[sb][4 * g + j];
-                if (cj == 0) continue;
-                uint32_t bw[32];
-#pragma unroll
-                for (int q = 0; q < 32; q += 4) {
-                    const uint4 x = *reinterpret_cast<const uint4*>(swords + 32 * j + q);
-                    bw[q] = x.x; bw[q + 1] = x.y; bw[q + 2] = x.z; bw[q + 3] = x.w;
-                }
-                const int64_t row0 = (a0 + 4 * (int64_t)g + j) * 1024;
-                const int a = (int)(((uintptr_t)(out + gc) >> 2) & 3);
-                int cur = a;
-#pragma unroll
-                for (int q = 0; q < 8; ++q) {
-                    const int cq = __popc(bw[4 * q]) + __popc(bw[4 * q + 1]) + __popc(bw[4 * q + 2]) + __popc(bw[4 * q + 3]);
-                    int pre = cur;
-#pragma unroll
-                    for (int jj = 0; jj < 4; ++jj) {
-                        const uint32_t w = bw[4 * q + jj];
-                        const int f = (w >> lane) & 1u;
-                        const int r = __popc(w & lt);
-                        const int32_t row = (int32_t)(row0 + (4 * q + jj) * 32 + lane);
-                        if (MODE == 0) {
-                            if (f) sw[pre + r] = row;
-                        } else {
-                            const int sel_before = pre - cur + r;
-                            const int kx = f ? pre + r : cur + cq + (jj * 32 + lane - sel_before);
-                            sw[kx] = row;
-                        }
-                        pre += __popc(w);
-                    }
-                    cur += cq;
-                }
-                __syncwarp();
-                const int tot = cur - a;
-                const int ngr = (a + tot + 3) >> 2;
-                int32_t* ob = out + gc - a;
-                for (int v = lane; v < ngr; v += 32) {
-                    const int4 x = *reinterpret_cast<const int4*>(sw + 4 * v);
-                    if (4 * v >= a && 4 * v + 4 <= a + tot) {
-                        __stcs(reinterpret_cast<int4*>(ob) + v, x);
-                    } else {
-                        const int32_t xs[4] = {x.x, x.y, x.z, x.w};
-#pragma unroll
-                        for (int e = 0; e < 4; ++e) {
-                            const int kx = 4 * v + e;
-                            if (kx >= a && kx < a + tot) __stcs(ob + kx, xs[e]);
-                        }
-                    }
-                }
-                __syncwarp();
-                gc += cj;
-            }
-        }
-        bar_sync_n(2, DEC * 32);  // every decoder done with the stripe's shared state
-        if (lane == 0) mbar_arrive(&H.freed[sb]);
-    }
-}
-
-static size_t sel_stream_smem(size_t tsize) {
-    return (size_t)SS_STG_N * SS_CPT * 1024 * tsize + (size_t)SS_DEC_MAX * SC_STG * 4 + sizeof(SsShared);
-}
-
-
-// VD_SELECT_STREAM_CNT (4, 6, 8): counting warps of the 15 (tuning runs)
-static int sel_stream_cnt() {
-    const char* e = getenv("VD_SELECT_STREAM_CNT");
-    const int x = e ? atoi(e) : 4;
-    return (x == 6 || x == 8) ? x : 4;
-}
-
-template <int MODE, typename T>
-static cudaError_t run_select_stream(const T* col, T lo, T hi, int64_t n, int32_t* out_pos, int64_t* out_count,
-                                     void* ws, cudaStream_t s, int* nl) {
-    if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
-    const int64_t nchunks = (n + 1023) / 1024;
-    const size_t sm = sel_stream_smem(sizeof(T));
-    const int cnt = sel_stream_cnt();
-    auto kern = cnt == 8 ? k_sel_stream<MODE, T, 8> : cnt == 6 ? k_sel_stream<MODE, T, 6> : k_sel_stream<MODE, T, 4>;
-    cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
-    int per_sm = 0;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SS_THREADS, sm) != cudaSuccess || per_sm < 1)
-        return cudaErrorNotSupported;
-    const int G = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, 4096);
-    // stripes: enough that one stripe's decode is a small tail, few enough
-    // that every (stripe, CTA) sub-range is several tiles
-    int S = (int)std::min<int64_t>(SS_MAXS, std::max<int64_t>(1, nchunks / ((int64_t)G * 64)));
-    while (S > 1 && (nchunks / S) / G + 2 > SS_MAXKB) --S;
-    if ((nchunks / S) / G + 2 > SS_MAXKB) return cudaErrorNotSupported;  // caller falls back
-    if (nchunks < (int64_t)G * 4) return cudaErrorNotSupported;          // small inputs: the single-barrier kernel
-    char* w = (char*)ws;
-    unsigned int* arrive = (unsigned int*)w;                              // [SS_MAXS]
-    int64_t* counts = (int64_t*)(w + 256);                                // [S][G]
-    uint32_t* bits = (uint32_t*)(w + 256 + al256((size_t)SS_MAXS * 4096 * 8));
-    cudaError_t e = cudaMemsetAsync(arrive, 0, SS_MAXS * 4, s);
-    if (e != cudaSuccess) return e;
-    static const int rmax = [] {
-        const char* v = getenv("VD_SELECT_ROUND_MAX");
-        const int x = v ? atoi(v) : SC_ROUND;
-        return x < 0 ? 0 : (x > SC_ROUND ? SC_ROUND : x);
-    }();
-    int round_max = rmax;
-    void* args[] = {(void*)&col, (void*)&lo, (void*)&hi, (void*)&n, (void*)&S, (void*)&out_pos, (void*)&out_count,
-                    (void*)&bits, (void*)&counts, (void*)&arrive, (void*)&round_max};
-    e = cudaLaunchCooperativeKernel((const void*)kern, dim3(G), dim3(SS_THREADS), args, sm, s);
-    ++*nl;
-    return e;
-}
-static size_t sel_stream_ws_bytes(int64_t n) {
-    const int64_t nchunks = (n + 1023) / 1024;
-    return 256 + al256((size_t)SS_MAXS * 4096 * 8) + al256((size_t)nchunks * 32 * 4);
-}
 
 // Per-row predicates (several columns, run heads): ballot j is word j.
 template <class F>
@@ -1534,42 +1111,57 @@ static cudaError_t run_select_bitmap(LaunchBits launch_bits, int64_t n, int32_t*
     return cudaGetLastError();
 }
 
-// ---- lagged single-pass selection: counts published, decode SL_LAG tiles later ----
-// One cooperative persistent kernel, one CTA per SM: a producer warp streams
-// tiles t = k*G + blockIdx (SL_CW 1024-row chunks each, round robin over the
-// grid) through a TMA ring; consumer warp w, in iteration k,
-//   counts    chunk w of tile k: 32 ballots -> one row-ordered bitmap word per
-//             lane, kept in REGISTERS (a queue of SL_LAG words per lane: the
-//             predicate materialised, Fig 8's break, never written to HBM);
-//             the chunk count goes to shared memory and, once per tile, the
-//             tile's count to a global table cnt[k][blockIdx];
-//   decodes   chunk w of tile k - SL_LAG, whose output base -- the counts of
-//             every earlier tile: all of rows < k - SL_LAG of the table plus
-//             the earlier CTAs of row k - SL_LAG -- one rotating warp per
-//             iteration read from the table (SL_LAG - 1 iterations after
-//             every CTA published it, so the loads rarely wait).
-// Reads of tile k and position writes of tile k - SL_LAG overlap inside every
-// SM, with no grid barrier, no look-back chain (a base is a sum over a row
-// the CTA reads whole) and no bitmap round trip through L2: k_sel_coop's
-// decode runs only after its grid barrier (HBM idle on reads meanwhile), the
-// striped k_sel_stream splits warps between counting and decoding.
-// Deadlock-free under a cooperative launch: row j of the table is published
-// by every CTA before it waits on any row (row j - SL_LAG + 1 < j).
+// ---- lagged single-pass selection (default for single interval terms on aligned 4-byte columns) ----
+// One cooperative persistent kernel, one CTA per SM; tile t = k*G + blockIdx
+// (SL_CW 1024-row chunks each, round robin over the grid):
+//   producer warp   in iteration k: loads tile k through a TMA ring (lane 0);
+//                   publishes tile k - SL_PUB (its chunk offsets to shared
+//                   memory, its count to a global table cnt[k][blockIdx]);
+//                   computes the output base of tile k - SL_BASE = the sum of
+//                   every earlier table row (a running total) + the earlier
+//                   CTAs' entries of its row, all published SL_BASE - SL_PUB
+//                   iterations before -- a row is read whole, no look-back chain;
+//   consumer warp w counts chunk w of tile k (lane L builds the bitmap word
+//                   of rows 32L..32L+31 out of the TMA stage: the predicate
+//                   materialised, Fig 8's break, kept in a per-lane REGISTER
+//                   queue of LAG words, never written to memory), then decodes
+//                   chunk w of tile k - LAG + 1 (positions staged in shared
+//                   memory, 16-byte stores).
+// Handoffs are mbarriers (counted[slot]: the SL_CW chunk counts; ready[slot]:
+// offsets + base), so no warp waits on the CTA's other warps per iteration,
+// and reads of tile k overlap position writes of tile k - LAG + 1 in every
+// SM.  k_sel_coop (below) decodes only after a grid barrier; a striped
+// counting/decoding warp split (k_sel_stream, round 2) and a per-iteration
+// CTA barrier instead of mbarriers were measured slower.
+// Deadlock-free under a cooperative launch: producer iteration k depends only
+// on producer iterations < k of every CTA (row k - SL_BASE is published at
+// iteration k - SL_BASE + SL_PUB), and consumers only on their producer.
 constexpr int SL_CW = 15;                     // consumer warps = chunks per tile
 constexpr int SL_THREADS = (SL_CW + 1) * 32;  // + the producer warp
-constexpr int SL_STAGES = 2;                  // 2 x 60 KB in flight per SM
-constexpr int SL_NS = 8;                      // per-tile shared slots (>= SL_LAG + 2)
-constexpr int SL_LAG = 3;                     // iterations between counting and decoding a tile
-constexpr int SL_STG = 1024 + 32 + 128 + 8;   // per-warp position stage (ints): chunk + pad + garbage
-constexpr int SL_SPARSE = 48;                 // default: branching chunks this sparse store directly,
-constexpr int SL_MID = 320;                   // ... this sparse: lane-owned rows, staged (VD_SEL_SPARSE / VD_SEL_MID)
+constexpr int SL_STAGES = 3;                  // 3 x 60 KB in flight per SM
+constexpr int SL_NS = 32;                     // per-tile shared slots (>= LAG + SL_STAGES + 1)
+constexpr int SL_LAG = 12;                    // default LAG: iterations between counting and decoding a tile
+                                              // (VD_SEL_LAG=16: a longer-lag instance)
+constexpr int SL_PUB = 2;                     // producer: publishes tile k - SL_PUB in iteration k
+constexpr int SL_BASE = 8;                    // ... and computes the base of tile k - SL_BASE
+constexpr int SL_STG = 512 + 128 + 60;        // per-warp position stage (ints): half a chunk + garbage, or
+                                              // VD_SEL_MID lane-owned positions + pad; the last 32: the words
+static_assert(3 + 512 + 128 + 4 <= SL_STG - 32, "dense stage");
+constexpr int SL_SPARSE = 48;                 // defaults: branching chunks this sparse store directly,
+constexpr int SL_MID = 320;                   // ... this sparse: lane-owned rows, staged;
+constexpr int SL_MID_PRED = 640;              // predicated chunks this sparse: lane-owned cursor arithmetic
+                                              // (VD_SEL_SPARSE / VD_SEL_MID override; measured at s = 0.5:
+                                              // predicated 0.89 ms lane-owned vs 1.05 ms ballot blocks,
+                                              // branching 0.97 either way)
+static_assert(640 + 4 + (640 + 4) / 32 + 4 <= SL_STG - 32, "lane-owned stage (VD_SEL_MID <= 640)");
 
 struct SlShared {
     uint64_t full[SL_STAGES], empty[SL_STAGES];
-    int cc[SL_NS][16];   // chunk counts of the tile in slot k % SL_NS
-    int off[SL_NS][16];  // their exclusive prefix within the tile
+    uint64_t counted[SL_NS];  // per slot: the SL_CW chunk counts are in cc
+    uint64_t ready[SL_NS];    // per slot: off (producer, publish) and base (producer, table row) are set
+    uint16_t cc[SL_NS][16];   // chunk counts of the tile in slot k % SL_NS
+    uint16_t off[SL_NS][16];  // their exclusive prefix within the tile
     int64_t base[SL_NS]; // the tile's output base
-    int64_t run;         // total of the table rows read so far
 };
 
 __device__ __forceinline__ uint32_t ld_relaxed_u32(const unsigned int* p) {
@@ -1579,6 +1171,21 @@ __device__ __forceinline__ uint32_t ld_relaxed_u32(const unsigned int* p) {
 }
 __device__ __forceinline__ void st_relaxed_u32(unsigned int* p, uint32_t v) {
     asm volatile("st.relaxed.gpu.global.u32 [%0], %1;" ::"l"(p), "r"(v) : "memory");
+}
+
+// `bit` if lo <= x <= hi (NaN / INT_MIN never: A9), else 0 -- two compares
+// into one predicate and one select
+__device__ __forceinline__ uint32_t ivl_bit(float x, float lo, float hi, uint32_t bit) {
+    uint32_t r;
+    asm("{\n\t.reg .pred p;\n\tsetp.ge.f32 p, %1, %2;\n\tsetp.le.and.f32 p, %1, %3, p;\n\tselp.b32 %0, %4, 0, p;\n\t}"
+        : "=r"(r) : "f"(x), "f"(lo), "f"(hi), "r"(bit));
+    return r;
+}
+__device__ __forceinline__ uint32_t ivl_bit(int32_t x, int32_t lo, int32_t hi, uint32_t bit) {
+    uint32_t r;
+    asm("{\n\t.reg .pred p;\n\tsetp.ge.s32 p, %1, %2;\n\tsetp.le.and.s32 p, %1, %3, p;\n\tselp.b32 %0, %4, 0, p;\n\t}"
+        : "=r"(r) : "r"(x), "r"(lo), "r"(hi), "r"(bit));
+    return r;
 }
 
 // Flush stage[a, a + tot) to o[0, tot) (o - a is 16-byte aligned): 16-byte
@@ -1685,14 +1292,18 @@ __device__ __forceinline__ void sl_decode(uint32_t word, int cnt, int32_t* __res
     // lane L places row 32j + L at the running rank (branching: qualifying
     // lanes only; predicated: cursor arithmetic -- every lane stores, rows that
     // do not qualify past the 128-row block's count, overwritten later)
+    const int32_t rl = row0 + lane;
+    uint32_t* ww = reinterpret_cast<uint32_t*>(sw + SL_STG - 32);  // the chunk's words, read back as broadcasts
+    ww[lane] = word;
+    __syncwarp();
+#pragma unroll
+    for (int h = 0; h < 2; ++h) {  // two 512-row halves, each staged and flushed
     const int a = (int)(((uintptr_t)o >> 2) & 3);
     int cur = a;
-    const int32_t rl = row0 + lane;
 #pragma unroll
-    for (int q = 0; q < 8; ++q) {
-        uint32_t bw[4];
-#pragma unroll
-        for (int jj = 0; jj < 4; ++jj) bw[jj] = __shfl_sync(VD_FULL, word, 4 * q + jj);
+    for (int q = 4 * h; q < 4 * h + 4; ++q) {
+        const uint4 b4 = *reinterpret_cast<const uint4*>(ww + 4 * q);
+        const uint32_t bw[4] = {b4.x, b4.y, b4.z, b4.w};
         const int cq = __popc(bw[0]) + __popc(bw[1]) + __popc(bw[2]) + __popc(bw[3]);
         int pre = cur;
 #pragma unroll
@@ -1714,14 +1325,17 @@ __device__ __forceinline__ void sl_decode(uint32_t word, int cnt, int32_t* __res
     __syncwarp();
     sl_flush(sw, a, cur - a, o, lane);
     __syncwarp();
+    o += cur - a;
+    }
 }
 
-template <int MODE, typename T>
+template <int MODE, typename T, int LAG>
 __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                            int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                            unsigned int* __restrict__ cnt /* [nk][G], zeroed */,
                                                            int sparse_max, int mid_max) {
     static_assert(sizeof(T) == 4, "k_sel_lag: 4-byte columns (f32 / i32)");
+    static_assert(SL_PUB < SL_BASE && SL_BASE < LAG && LAG + SL_STAGES + 1 <= SL_NS, "k_sel_lag: lags / shared slots");
     constexpr uint32_t TB = SL_CW * 1024 * sizeof(T);
     extern __shared__ __align__(128) uint8_t smem[];
     int32_t* stages = reinterpret_cast<int32_t*>(smem + (size_t)SL_STAGES * TB);
@@ -1736,73 +1350,129 @@ __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__
             mbar_init(&H.full[i], 1);
             mbar_init(&H.empty[i], SL_CW);
         }
-        H.run = 0;
+        for (int i = 0; i < SL_NS; ++i) {
+            mbar_init(&H.counted[i], SL_CW);
+            mbar_init(&H.ready[i], 2);
+        }
         fence_mbar_init();
     }
     __syncthreads();
-    if (warp == SL_CW) {  // producer
-        if (lane == 0) {
-            const uint64_t pol = policy_evict_first();
-            int st = 0;
-            uint32_t ph = 0;
-            for (int64_t k = 0; k < myk; ++k) {
-                if (k >= SL_STAGES) mbar_wait(&H.empty[st], ph ^ 1u);
-                const int64_t r0 = (k * G + c) * (int64_t)SL_CW * 1024;
-                if (r0 + (int64_t)SL_CW * 1024 <= n) {
-                    mbar_expect_tx(&H.full[st], TB);
-                    tma_load_1d(smem + (size_t)st * TB, col + r0, TB, &H.full[st], pol);
-                } else {
-                    mbar_arrive(&H.full[st]);  // the column's last, partial tile: consumers load it directly
+    if (warp == SL_CW) {
+        // ---- producer / bookkeeping warp: in iteration k it
+        //   loads tile k (lane 0, TMA),
+        //   publishes tile k - SL_PUB: chunk offsets to shared memory, the
+        //     tile's count to the table,
+        //   computes the base of tile k - SL_BASE from table row k - SL_BASE
+        //     (published by every CTA SL_BASE - SL_PUB iterations earlier),
+        // and the two halves of ready[tile] let its decoders go.
+        const uint64_t pol = policy_evict_first();
+        int st = 0;
+        uint32_t ph = 0;
+        int64_t run = 0;  // the totals of the rows read so far
+        for (int64_t k = 0; k < myk + SL_BASE; ++k) {
+            if (k < myk) {
+                if (lane == 0) {
+                    if (k >= SL_STAGES) mbar_wait(&H.empty[st], ph ^ 1u);
+                    const int64_t r0 = (k * G + c) * (int64_t)SL_CW * 1024;
+                    if (r0 + (int64_t)SL_CW * 1024 <= n) {
+                        mbar_expect_tx(&H.full[st], TB);
+                        tma_load_1d(smem + (size_t)st * TB, col + r0, TB, &H.full[st], pol);
+                    } else {
+                        mbar_arrive(&H.full[st]);  // the column's last, partial tile: consumers load it directly
+                    }
                 }
                 if (++st == SL_STAGES) { st = 0; ph ^= 1u; }
+                __syncwarp();
+            }
+            const int64_t kp = k - SL_PUB;
+            if (kp >= 0 && kp < myk) {
+                const int sp = (int)(kp & (SL_NS - 1));
+                mbar_wait(&H.counted[sp], (uint32_t)(kp / SL_NS) & 1u);
+                const int x = lane < SL_CW ? H.cc[sp][lane] : 0;
+                int incl = x;
+#pragma unroll
+                for (int d = 1; d < 32; d <<= 1) {
+                    const int u = __shfl_up_sync(VD_FULL, incl, d);
+                    if (lane >= d) incl += u;
+                }
+                if (lane < SL_CW) H.off[sp][lane] = (uint16_t)(incl - x);
+                if (lane == 31) st_relaxed_u32(cnt + kp * G + c, (uint32_t)incl + 1u);
+                __syncwarp();
+                if (lane == 0) mbar_arrive(&H.ready[sp]);
+            }
+            const int64_t kb = k - SL_BASE;
+            if (kb >= 0 && kb < myk) {
+                uint32_t rv[5];
+#pragma unroll
+                for (int i = 0; i < 5; ++i) {
+                    const int j = lane + 32 * i;
+                    rv[i] = (j < G && kb * G + j < ntiles) ? ld_relaxed_u32(cnt + kb * G + j) : 1u;  // absent: 0
+                }
+                int pre = 0, tot = 0;
+#pragma unroll
+                for (int i = 0; i < 5; ++i) {
+                    const int j = lane + 32 * i;
+                    while (rv[i] == 0u) {
+                        __nanosleep(20);
+                        rv[i] = ld_relaxed_u32(cnt + kb * G + j);
+                    }
+                    const int x = (int)rv[i] - 1;
+                    tot += x;
+                    pre += j < c ? x : 0;
+                }
+#pragma unroll
+                for (int d = 16; d; d >>= 1) {
+                    pre += __shfl_xor_sync(VD_FULL, pre, d);
+                    tot += __shfl_xor_sync(VD_FULL, tot, d);
+                }
+                const int sb = (int)(kb & (SL_NS - 1));
+                if (lane == 0) {
+                    H.base[sb] = run + pre;
+                    mbar_arrive(&H.ready[sb]);
+                }
+                run += tot;
             }
         }
+        // CTA 0 owns a tile in every row: its run is the grand total
+        if (c == 0 && lane == 0) *out_count = run;
         return;
     }
+    // ---- consumer warps: count chunk `warp` of tile k, decode it LAG iterations later ----
     int32_t* sw = stages + warp * SL_STG;
-    uint32_t q[SL_LAG];
+    uint32_t q[LAG];
 #pragma unroll
-    for (int i = 0; i < SL_LAG; ++i) q[i] = 0;
-    int st = 0, rk = 0;  // rk = k % SL_CW
+    for (int i = 0; i < LAG; ++i) q[i] = 0;
+    int st = 0;
     uint32_t ph = 0;
-    for (int64_t k = 0; k < myk + SL_LAG; ++k, rk = rk + 1 == SL_CW ? 0 : rk + 1) {
-        const int slot = (int)(k & (SL_NS - 1));
-        // (A) this iteration's base warp issues the loads of table row kb
-        const int64_t kb = k - SL_LAG + 1;
-        const bool role = warp == rk && kb >= 0 && kb < myk;
-        uint32_t rv[5];
-        if (role) {
-#pragma unroll
-            for (int i = 0; i < 5; ++i) {
-                const int j = lane + 32 * i;
-                rv[i] = (j < G && kb * G + j < ntiles) ? ld_relaxed_u32(cnt + kb * G + j) : 1u;  // absent tile: count 0
-            }
-        }
-        // (B) count chunk `warp` of tile k
-        uint32_t word = 0;
+    for (int64_t k = 0; k < myk + LAG; ++k) {
         if (k < myk) {
+            const int slot = (int)(k & (SL_NS - 1));
+            uint32_t word = 0;
             mbar_wait(&H.full[st], ph);
             const int64_t t = k * G + c;
             const int64_t ch = t * SL_CW + warp;
             if (ch < nchunks) {
                 if ((t + 1) * (int64_t)SL_CW * 1024 <= n) {
-                    const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024;
+                    // lane L: rows 32L .. 32L+31 of the chunk in 8 16-byte loads,
+                    // rotated by L so the 8 lanes of a load phase hit 8
+                    // different 16-byte bank groups (conflict-free)
+                    const T* src = reinterpret_cast<const T*>(smem + (size_t)st * TB) + warp * 1024 + 32 * lane;
 #pragma unroll
-                    for (int j = 0; j < 32; ++j) {
-                        const T v = src[j * 32 + lane];
-                        const uint32_t b = __ballot_sync(VD_FULL, v >= lo && v <= hi);  // NaN / INT_MIN fail
-                        word = lane == j ? b : word;
+                    for (int m = 0; m < 8; ++m) {
+                        const int mm = (m + lane) & 7;
+                        T x[4];
+                        Vec4Lds<T>::ld(src + 4 * mm, x);
+                        const uint32_t nib = ivl_bit(x[0], lo, hi, 1u) | ivl_bit(x[1], lo, hi, 2u) |
+                                             ivl_bit(x[2], lo, hi, 4u) | ivl_bit(x[3], lo, hi, 8u);
+                        word |= nib << (4 * mm);
                     }
                 } else {
-                    for (int j = 0; j < 32; ++j) {
-                        const int64_t r = ch * 1024 + j * 32 + lane;
-                        bool f = false;
+                    for (int i = 0; i < 32; ++i) {
+                        const int64_t r = ch * 1024 + 32 * lane + i;
                         if (r < n) {
                             const T v = __ldg(col + r);
-                            f = v >= lo && v <= hi;
+                            word |= (uint32_t)(v >= lo && v <= hi) << i;
                         }
-                        const uint32_t b = __ballot_sync(VD_FULL, f);
-                        word = lane == j ? b : word;
                     }
                 }
             }
@@ -1812,49 +1482,23 @@ __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__
             int cw = __popc(word);
 #pragma unroll
             for (int d = 16; d; d >>= 1) cw += __shfl_xor_sync(VD_FULL, cw, d);
-            if (lane == 0) H.cc[slot][warp] = cw;
-        }
-        // (C) base of tile kb: the earlier rows' totals + the earlier CTAs of row kb
-        if (role) {
-            int pre = 0, tot = 0;
-#pragma unroll
-            for (int i = 0; i < 5; ++i) {
-                const int j = lane + 32 * i;
-                while (rv[i] == 0u) {
-                    __nanosleep(32);
-                    rv[i] = ld_relaxed_u32(cnt + kb * G + j);
-                }
-                const int x = (int)rv[i] - 1;
-                tot += x;
-                pre += j < c ? x : 0;
-            }
-#pragma unroll
-            for (int d = 16; d; d >>= 1) {
-                pre += __shfl_xor_sync(VD_FULL, pre, d);
-                tot += __shfl_xor_sync(VD_FULL, tot, d);
-            }
             if (lane == 0) {
-                H.base[kb & (SL_NS - 1)] = H.run + pre;
-                H.run += tot;
+                H.cc[slot][warp] = (uint16_t)cw;
+                mbar_arrive(&H.counted[slot]);  // release: the count is visible to the producer's wait
             }
-        }
-        bar_sync_n(1, SL_CW * 32);
-        // (D) publish tile k: chunk offsets to shared memory, its count to the table
-        if (k < myk && warp == (rk + 7 < SL_CW ? rk + 7 : rk + 7 - SL_CW)) {
-            const int x = lane < SL_CW ? H.cc[slot][lane] : 0;
-            int incl = x;
 #pragma unroll
-            for (int d = 1; d < 32; d <<= 1) {
-                const int u = __shfl_up_sync(VD_FULL, incl, d);
-                if (lane >= d) incl += u;
-            }
-            if (lane < SL_CW) H.off[slot][lane] = incl - x;
-            if (lane == 31) st_relaxed_u32(cnt + k * G + c, (uint32_t)incl + 1u);
+            for (int i = 0; i + 1 < LAG; ++i) q[i] = q[i + 1];
+            q[LAG - 1] = word;
+        } else {
+#pragma unroll
+            for (int i = 0; i + 1 < LAG; ++i) q[i] = q[i + 1];
+            q[LAG - 1] = 0;
         }
-        // (E) decode chunk `warp` of tile k - SL_LAG
-        const int64_t kd = k - SL_LAG;
-        if (kd >= 0) {
+        // decode chunk `warp` of tile k - LAG + 1 (q[0])
+        const int64_t kd = k - LAG + 1;
+        if (kd >= 0 && kd < myk) {
             const int ds = (int)(kd & (SL_NS - 1));
+            mbar_wait(&H.ready[ds], (uint32_t)(kd / SL_NS) & 1u);
             const int cd = H.cc[ds][warp];
             if (cd > 0) {
                 const int64_t ob = H.base[ds] + H.off[ds][warp];
@@ -1862,13 +1506,6 @@ __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__
                 sl_decode<MODE>(q[0], cd, out + ob, row0, sw, lane, sparse_max, mid_max);
             }
         }
-#pragma unroll
-        for (int i = 0; i + 1 < SL_LAG; ++i) q[i] = q[i + 1];
-        q[SL_LAG - 1] = word;
-    }
-    if (c == 0) {
-        bar_sync_n(1, SL_CW * 32);
-        if (threadIdx.x == 0) *out_count = H.run;
     }
 }
 
@@ -1880,13 +1517,11 @@ static size_t sel_lag_ws_bytes(int64_t n) {
     return al256((size_t)(ntiles + 4096) * 4);
 }
 
-// VD_SELECT_KERNEL=coop / stream: the single-barrier or striped kernel instead
-// (comparison runs; read per call: tests switch kernels inside one process)
+// VD_SELECT_KERNEL=coop: the single-barrier kernel instead (comparison runs;
+// read per call: tests switch kernels inside one process)
 static int sel_kernel_choice() {
     const char* e = getenv("VD_SELECT_KERNEL");
-    if (e && strcmp(e, "coop") == 0) return 1;
-    if (e && strcmp(e, "stream") == 0) return 2;
-    return 0;
+    return (e && strcmp(e, "coop") == 0) ? 1 : 0;
 }
 
 template <int MODE, typename T>
@@ -1895,7 +1530,8 @@ static cudaError_t run_select_lag(const T* col, T lo, T hi, int64_t n, int32_t* 
     if (n == 0) return cudaMemsetAsync(out_count, 0, sizeof(int64_t), s);
     const int64_t ntiles = ((n + 1023) / 1024 + SL_CW - 1) / SL_CW;
     const size_t sm = sel_lag_smem();
-    auto kern = k_sel_lag<MODE, T>;
+    const char* lv = getenv("VD_SEL_LAG");
+    auto kern = (lv && atoi(lv) == 16) ? k_sel_lag<MODE, T, 16> : k_sel_lag<MODE, T, SL_LAG>;
     cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sm);
     int per_sm = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SL_THREADS, sm) != cudaSuccess || per_sm < 1)
@@ -1912,7 +1548,8 @@ static cudaError_t run_select_lag(const T* col, T lo, T hi, int64_t n, int32_t* 
         const int x = v ? atoi(v) : dflt;
         return x < 0 ? 0 : (x > hi ? hi : x);
     };
-    int sparse_max = knob("VD_SEL_SPARSE", SL_SPARSE, 1024), mid_max = knob("VD_SEL_MID", SL_MID, 1024);
+    // lane-owned chunks must fit the stage: x + x/32 + 4 < SL_STG
+    int sparse_max = knob("VD_SEL_SPARSE", SL_SPARSE, 1024), mid_max = knob("VD_SEL_MID", MODE ? SL_MID_PRED : SL_MID, 640);
     void* args[] = {(void*)&col,       (void*)&lo,  (void*)&hi,         (void*)&n,      (void*)&out_pos,
                     (void*)&out_count, (void*)&cnt, (void*)&sparse_max, (void*)&mid_max};
     e = cudaLaunchCooperativeKernel((const void*)kern, dim3(G), dim3(SL_THREADS), args, sm, s);
@@ -1924,7 +1561,7 @@ size_t select_ws_bytes(int64_t n) {
     int64_t ntiles = (n + SEL_TILE - 1) / SEL_TILE;
     size_t b = 256 + (size_t)ntiles * 8;
     size_t lb = (b + 255) & ~(size_t)255;
-    size_t bm = std::max(std::max(bm_ws_bytes(n), sel_lag_ws_bytes(n)), std::max(sel_coop_ws_bytes(n), sel_stream_ws_bytes(n)));
+    size_t bm = std::max(std::max(bm_ws_bytes(n), sel_lag_ws_bytes(n)), sel_coop_ws_bytes(n));
     return lb > bm ? lb : bm;
 }
 
@@ -2026,10 +1663,6 @@ static cudaError_t dispatch_term(const void* p, const DevTerm& t, int64_t n, int
                     set_fragment("sel_lag");
                     cudaError_t e = run_select_lag<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
                     if (e != cudaErrorNotSupported) return e;  // else: small, the single-barrier kernel
-                } else if (kc == 2) {
-                    set_fragment("sel_stream");
-                    cudaError_t e = run_select_stream<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);
-                    if (e != cudaErrorNotSupported) return e;  // else: small / too large, the single-barrier kernel
                 }
                 set_fragment("sel_coop");
                 cudaError_t e = run_select_coop<MODE, T>((const T*)p, ilo, ihi, n, out_pos, out_count, ws, s, nl);

@@ -1,0 +1,9 @@
+# Round 2 (re-entry 3): k_sel_lag v2 (rotated 16-byte count loads, 3-stage ring, half-chunk dense flush)
+set -x
+mkdir -p gpurun_out
+timeout 1200 python -m pytest tests/test_gpu_select_coop.py -m gpu -q -x -p no:cacheprovider > gpurun_out/r2z_pytest.log 2>&1; echo "rc=$?" >> gpurun_out/r2z_pytest.log
+for s in 0.0001 0.01 0.1 0.5 1.0; do for m in branch predicated; do
+  timeout 300 python bench.py --workload selpos --selectivity $s --sel-mode $m --steps 30 --no-cpu-baseline 2>> gpurun_out/r2z_bench.err | sed "s/^/lag /" >> gpurun_out/r2z_selpos.txt
+done; done
+timeout 600 ncu --set full --clock-control none --import-source on -k regex:k_sel_lag -s 2 -c 1 -o gpurun_out/r2z_prof_lag05 -f python bench.py --workload selpos --selectivity 0.5 --steps 2 --warmup 2 --no-cpu-baseline > gpurun_out/r2z_ncu.log 2>&1
+timeout 600 ncu --set full --clock-control none --import-source on -k regex:k_sel_lag -s 2 -c 1 -o gpurun_out/r2z_prof_lag0001 -f python bench.py --workload selpos --selectivity 0.0001 --steps 2 --warmup 2 --no-cpu-baseline >> gpurun_out/r2z_ncu.log 2>&1

@@ -85,16 +85,15 @@ def test_fused_select_i32_tiles_alternating_empty_and_full(mode):
 
 
 @pytest.mark.parametrize("mode", ["branch", "predicated"])
-@pytest.mark.parametrize("n,t", [(5 * 10**6 + 3, 0.3), (50 * 10**6 + 17, 0.02), (50 * 10**6 + 17, 0.7),
+@pytest.mark.parametrize("n,t", [(10 * 10**6 + 3, 0.3), (50 * 10**6 + 17, 0.02), (50 * 10**6 + 17, 0.7),
                                  (120 * 10**6 + 1, 0.5), (37 * 10**6 + 4093, 0.002), (41 * 10**6 + 9, 0.12)])
 def test_large_select_kernels_vs_oracle(mode, n, t):
     """The large-input kernels against the oracle's brute-force selection:
     the default lagged single pass (k_sel_lag: tile counts published to a
-    table, each tile decoded SL_LAG iterations later from register-held
-    words; sparse / lane-owned / dense chunk paths), the striped
-    warp-specialised kernel (k_sel_stream) and the single-barrier kernel
-    (k_sel_coop), at sizes with a ragged last tile, into an unaligned
-    output."""
+    table, each tile decoded LAG iterations later from register-held words;
+    sparse / lane-owned / dense chunk paths) at both compiled lags, and the
+    single-barrier kernel (k_sel_coop), at sizes with a ragged last tile,
+    into an unaligned output."""
     v = gen.host(gen.F32_UNIFORM, n, seed=n % 1009)
     t = float(np.float32(t))
     pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
@@ -103,17 +102,22 @@ def test_large_select_kernels_vs_oracle(mode, n, t):
     got = _select(fn, dv, n, t, shift=1)
     assert vd.last_fragment() == "sel_lag"
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
-    for kern in ("stream", "coop"):
-        with env(VD_SELECT_KERNEL=kern):
-            assert np.array_equal(_select(fn, dv, n, t), pos_o)
-            assert vd.last_fragment() == "sel_" + kern
+    with env(VD_SEL_LAG="16"):
+        assert np.array_equal(_select(fn, dv, n, t), pos_o)
+        assert vd.last_fragment() == "sel_lag"
+    with env(VD_SELECT_KERNEL="coop"):
+        assert np.array_equal(_select(fn, dv, n, t), pos_o)
+        assert vd.last_fragment() == "sel_coop"
 
 
 @pytest.mark.parametrize("mode", ["branch", "predicated"])
-def test_lag_select_chunk_density_mix(mode):
+@pytest.mark.parametrize("mid", [None, "0", "640"])
+def test_lag_select_chunk_density_mix(mode, mid):
     """Chunks of every density class of k_sel_lag's decode in one input
-    (empty, <= SL_SPARSE, <= SL_MID, dense, full) with NaN epsilon rows,
-    i32 and f32, against the oracle."""
+    (empty, <= SL_SPARSE, lane-owned, dense ballot blocks, full) with NaN
+    epsilon rows, i32 and f32, against the oracle; the lane-owned threshold
+    at its default, off (every chunk through the ballot blocks) and at its
+    maximum."""
     n = 148 * 15 * 1024 * 6 + 12345
     rng = np.random.default_rng(7)
     chunk = np.arange(n) // 1024
@@ -122,6 +126,11 @@ def test_lag_select_chunk_density_mix(mode):
     v[::977] = np.nan
     pos_o, cnt_o, _ = oracle.select_f32(v, 0.5, "lt")
     fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    with env(**({} if mid is None else {"VD_SEL_MID": mid})):
+        _density_mix_check(fn, v, n, pos_o, cnt_o)
+
+
+def _density_mix_check(fn, v, n, pos_o, cnt_o):
     got = _select(fn, torch.from_numpy(v).cuda(), n, 0.5, shift=3)
     assert vd.last_fragment() == "sel_lag"
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
