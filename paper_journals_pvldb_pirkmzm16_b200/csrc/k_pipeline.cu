@@ -1621,7 +1621,11 @@ __device__ __forceinline__ int4 lt_ld16(const void* p, uint64_t pol) {
     return r;
 }
 
-template <int N8, bool I32>
+// CP: the predicate compiled to constraints / acceptance tables (ld.ncons[0]
+// >= 0, every plan without NE terms), else the term lists are interpreted --
+// one evaluator per instance keeps the drain's code within the instruction
+// cache
+template <int N8, bool I32, bool CP>
 __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_constant__ GfArgs a,
                                                          const __grid_constant__ LateLead ld,
                                                          Slot16* __restrict__ parts, unsigned int* __restrict__ done,
@@ -1647,11 +1651,10 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
     // the rest of the predicate and the aggregate inputs of one lead-qualified row
     auto fold_row = [&](int64_t row) {
         late_load(a, ld.pref1, row, s_v, tid, pol_s, pol_d);
-        const bool compiled = ld.ncons[0] >= 0;
-        int t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1, s_tab) : late_pred(a, s_v, tid, ld.pref1);
+        int t = CP ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1, s_tab) : late_pred(a, s_v, tid, ld.pref1);
         if (t == 2) {
             late_load(a, ld.pref & ~ld.pref1, row, s_v, tid, pol_s, pol_d);
-            t = compiled ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref, s_tab) : late_pred(a, s_v, tid, ld.pref);
+            t = CP ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref, s_tab) : late_pred(a, s_v, tid, ld.pref);
         }
         if (t != 1) return;
         late_load(a, ld.aref & ~ld.pref, row, s_v, tid, pol_s, pol_d);
@@ -4139,16 +4142,18 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
         // (the attribute is per device context: set on every launch, as for
         // the other dynamic-shared-memory fragments)
-#define LT_GO(N8_, I32_)                                                                                    \
+#define LT_GO1(N8_, I32_, CP_)                                                                              \
     do {                                                                                                    \
-        e = cudaFuncSetAttribute(k_pipe_late<N8_, I32_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
+        e = cudaFuncSetAttribute(k_pipe_late<N8_, I32_, CP_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }                     \
-        k_pipe_late<N8_, I32_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);               \
+        k_pipe_late<N8_, I32_, CP_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);          \
     } while (0)
+#define LT_GO(N8_, I32_) do { if (L.ncons[0] >= 0) LT_GO1(N8_, I32_, true); else LT_GO1(N8_, I32_, false); } while (0)
         if (n8 == 2) { if (i32) LT_GO(2, true); else LT_GO(2, false); }
         else if (n8 == 1) { if (i32) LT_GO(1, true); else LT_GO(1, false); }
         else LT_GO(0, true);
 #undef LT_GO
+#undef LT_GO1
         ++*nl;
         e = cudaGetLastError();
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
