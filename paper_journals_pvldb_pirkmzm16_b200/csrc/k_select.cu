@@ -1536,8 +1536,9 @@ static cudaError_t run_select_lag(const T* col, T lo, T hi, int64_t n, int32_t* 
     int per_sm = 0;
     if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, SL_THREADS, sm) != cudaSuccess || per_sm < 1)
         return cudaErrorNotSupported;
-    const int G = (int)std::min<int64_t>((int64_t)num_sms() * per_sm, 160);  // a table row = 5 loads per lane
-    if (ntiles < (int64_t)G * 4) return cudaErrorNotSupported;              // small inputs: the single-barrier kernel
+    // one CTA per SM, at most one per tile (small inputs: one tile each, the
+    // table a single row); a table row = 5 loads per lane
+    const int G = (int)std::min<int64_t>(std::min<int64_t>((int64_t)num_sms() * per_sm, 160), ntiles);
     if (n > (int64_t)INT32_MAX) return cudaErrorNotSupported;
     const int64_t nk = (ntiles + G - 1) / G;
     unsigned int* cnt = (unsigned int*)ws;

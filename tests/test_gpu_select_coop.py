@@ -1,4 +1,6 @@
-"""The single-launch selection kernel (k_sel_coop: per-CTA contiguous chunk
+"""The single-launch selection kernels (k_sel_lag, the default at every size:
+tiles counted into register-held words, counts published to a table, each
+tile decoded LAG iterations later; k_sel_coop: per-CTA contiguous chunk
 ranges streamed by TMA into ballot words, one grid barrier, in-order decode
 into staged 16-byte stores) against the oracle: sizes from one row to
 several 16-chunk tiles per CTA with a ragged end (TMA tiles, LDG for the
@@ -44,6 +46,10 @@ def test_fused_select_f32_vs_oracle(mode, n, t):
     dv = torch.from_numpy(v).cuda()
     got = _select(fn, dv, n, t)
     assert len(got) == cnt_o and np.array_equal(got, pos_o)
+    assert vd.last_fragment() == "sel_lag"
+    with env(VD_SELECT_KERNEL="coop"):  # the single-barrier kernel agrees
+        assert np.array_equal(_select(fn, dv, n, t), pos_o)
+        assert vd.last_fragment() == "sel_coop"
     with env(VD_SELECT_COOP="0"):  # the bitmap path agrees
         assert np.array_equal(_select(fn, dv, n, t), pos_o)
 
