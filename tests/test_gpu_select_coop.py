@@ -147,3 +147,67 @@ def _density_mix_check(fn, v, n, pos_o, cnt_o):
     assert vd.last_fragment() == "sel_lag"
     k = int(cnt.item())
     assert k == cnt_o and np.array_equal(out[:k].cpu().numpy(), pos_o)
+
+
+@pytest.mark.parametrize("mode", ["branch", "predicated"])
+@pytest.mark.parametrize("cmp,thr", [("<", -700), (">=", 250), ("==", 17), ("<=", 999)])
+def test_lag_select_i32_large_vs_interpreter(mode, cmp, thr):
+    """k_sel_lag on an int32 column of 12 M rows (several tiles per CTA, a
+    ragged last tile): negative values, epsilon (INT32_MIN, never selected:
+    A9), one-sided / equality / nearly-all predicates, against the oracle's
+    interpreter (comparison -> FoldSelect)."""
+    n = 12 * 10**6 + 777
+    rng = np.random.default_rng(4242 + thr)
+    a = rng.integers(-1000, 1000, n).astype(np.int32)
+    m = rng.random(n) < 0.003
+    a[m] = -2**31
+    prog = {"<": f"p := Greater({thr}, v)", ">=": f"p := Greater(v, {thr - 1})",
+            "==": f"p := Equals(v, {thr})", "<=": f"p := Greater({thr + 1}, v)"}[cmp]
+    res = oracle.run(prog + "\npos := FoldSelect(p)", v=(a.astype(np.int64), m))
+    pos, pe = res.get_arrays("pos")
+    exp = pos[~pe]
+    fn = vd.select_branch if mode == "branch" else vd.select_predicated
+    out = torch.full((n + 4,), -7, dtype=torch.int32, device="cuda")
+    cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+    fn([vd.column(torch.from_numpy(a).cuda())], n, vd.pred([[(0, cmp, thr)]]), out_pos=out[1:n + 1], out_count=cnt)
+    assert vd.last_fragment() == "sel_lag"
+    k = int(cnt.item())
+    assert k == exp.size and np.array_equal(out[1:k + 1].cpu().numpy(), exp)
+    assert out[0].item() == -7 and (k == n or out[k + 1].item() == -7)
+
+
+def test_lag_select_in_cuda_graph():
+    """k_sel_lag's launch (table memset + cooperative kernel) captured in a
+    CUDA graph and replayed: every replay equals the oracle, for two
+    thresholds captured in two graphs replayed alternately."""
+    n = 20 * 10**6 + 3
+    v = gen.host(gen.F32_UNIFORM, n, seed=77)
+    dv = torch.from_numpy(v).cuda()
+    graphs, outs, exps = [], [], []
+    side = torch.cuda.Stream()
+    side.wait_stream(torch.cuda.current_stream())
+    for t in (0.05, 0.6):
+        t = float(np.float32(t))
+        pos_o, cnt_o, _ = oracle.select_f32(v, t, "lt")
+        exps.append(pos_o)
+        out = torch.empty(n, dtype=torch.int32, device="cuda")
+        cnt = torch.zeros(1, dtype=torch.int64, device="cuda")
+        ws = vd.alloc_ws(vd.workspace_bytes(vd.VD_OP_SELECT, n), dv.device)
+        g = torch.cuda.CUDAGraph()
+        with torch.cuda.stream(side):
+            with torch.cuda.graph(g, stream=side):
+                vd.select_branch([vd.column(dv)], n, vd.pred([[(0, "<", t)]]), out_pos=out, out_count=cnt, ws=ws,
+                                 stream=side)
+        assert vd.last_fragment() == "sel_lag"
+        graphs.append(g)
+        outs.append((out, cnt, ws))
+    torch.cuda.current_stream().wait_stream(side)
+    torch.cuda.synchronize()
+    for rep in range(3):
+        for g, (out, cnt, _), exp in zip(graphs, outs, exps):
+            out.fill_(-1)
+            cnt.zero_()
+            g.replay()
+            torch.cuda.synchronize()
+            k = int(cnt.item())
+            assert k == exp.size and np.array_equal(out[:k].cpu().numpy(), exp), rep
