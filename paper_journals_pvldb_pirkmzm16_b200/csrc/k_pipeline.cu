@@ -1450,6 +1450,13 @@ struct LateLead {
     int32_t tref[4];
     uint32_t tcm[4];
     uint8_t tab[4][256];
+    // fast first round (PV == 2): the first-round references are one int32
+    // FK column and nfg u8 lookups through it whose every constraint is
+    // tabulated -- the loads go to registers and the tables decide at once
+    // whether any conjunction can still pass (most lead rows: none)
+    int32_t fk_col, nfg;
+    int32_t fg[VD_MAX_GATHERS];     // gather index of fast lookup j
+    int32_t fgtab[VD_MAX_GATHERS];  // its acceptance table
 };
 constexpr int LT_MAXTAB = 4;
 constexpr int LT_COMMON = 4;  // = VD_MAX_CONJ
@@ -1603,6 +1610,16 @@ __device__ __forceinline__ int late_pred_c(const LateLead& ld, int nconj, const 
     return yes ? 1 : 2;
 }
 
+__device__ __forceinline__ uint32_t ld64b_hint_u32(const void* p, uint64_t pol) {
+    uint32_t v;
+    asm volatile("ld.global.nc.L2::cache_hint.L2::64B.u32 %0, [%1], %2;" : "=r"(v) : "l"(p), "l"(pol));
+    return v;
+}
+__device__ __forceinline__ uint32_t ld64b_hint_u8(const void* p, uint64_t pol) {
+    uint16_t v;
+    asm volatile("ld.global.nc.L2::cache_hint.L2::64B.u8 %0, [%1], %2;" : "=h"(v) : "l"(p), "l"(pol));
+    return v;
+}
 __device__ __forceinline__ uint32_t lt_mask_i32(const int4 (&v)[4], int32_t lo, int32_t hi) {
     uint32_t m = 0;
 #pragma unroll
@@ -1621,11 +1638,11 @@ __device__ __forceinline__ int4 lt_ld16(const void* p, uint64_t pol) {
     return r;
 }
 
-// CP: the predicate compiled to constraints / acceptance tables (ld.ncons[0]
-// >= 0, every plan without NE terms), else the term lists are interpreted --
-// one evaluator per instance keeps the drain's code within the instruction
-// cache
-template <int N8, bool I32, bool CP>
+// PV: the predicate evaluator -- 0: the term lists interpreted; 1: compiled
+// to constraints / acceptance tables (ld.ncons[0] >= 0, every plan without
+// NE terms); 2: compiled, with the fast first round (ld.nfg > 0).  One
+// evaluator per instance keeps the drain's code within the instruction cache
+template <int N8, bool I32, int PV>
 __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_constant__ GfArgs a,
                                                          const __grid_constant__ LateLead ld,
                                                          Slot16* __restrict__ parts, unsigned int* __restrict__ done,
@@ -1649,8 +1666,10 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
     int cnt = 0;  // warp-uniform queue depth
     for (int g = 0; g <= NA; ++g) s_a[g][tid] = 0;
     // the rest of the predicate and the aggregate inputs of one lead-qualified row
-    auto fold_row = [&](int64_t row) {
-        late_load(a, ld.pref1, row, s_v, tid, pol_s, pol_d);
+    constexpr bool CP = PV >= 1;
+    // everything after the first round (its references in s_v): the rest of
+    // the predicate, the undecided rows' second round, the aggregate inputs
+    auto rest_row = [&](int64_t row) {
         int t = CP ? late_pred_c(ld, a.pred.nconj, s_v, tid, ld.pref1, s_tab) : late_pred(a, s_v, tid, ld.pref1);
         if (t == 2) {
             late_load(a, ld.pref & ~ld.pref1, row, s_v, tid, pol_s, pol_d);
@@ -1677,6 +1696,32 @@ __global__ void __launch_bounds__(LT_THREADS, 4) k_pipe_late(const __grid_consta
             s_a[g][tid] += pr;
         }
         s_a[NA][tid] += 1;
+    };
+    auto fold_row = [&](int64_t row) {
+        if (PV == 2) {
+            // the FK and the lookups straight to registers (also kept in s_v
+            // for the later rounds), the tables ANDed: reject at once unless
+            // a conjunction (and the common terms) can still pass (most lead
+            // rows: none)
+            const int32_t fk = (int32_t)ld64b_hint_u32((const int32_t*)a.col[ld.fk_col] + row, pol_s);
+            s_v[ld.fk_col][tid] = fk == INT32_MIN ? INT64_MIN : (int64_t)fk;
+            uint32_t m = ((1u << a.pred.nconj) - 1) | (1u << LT_COMMON);
+#pragma unroll
+            for (int j = 0; j < VD_MAX_GATHERS; ++j) {
+                if (j >= ld.nfg) break;
+                const int g = ld.fg[j];
+                const int64_t pidx = (int64_t)fk - a.g_bias[g];
+                uint32_t x = 0xFFu;
+                if (fk != INT32_MIN && pidx >= 0 && pidx < a.g_len[g])
+                    x = ld64b_hint_u8((const uint8_t*)a.g_p[g] + pidx, pol_d);
+                s_v[a.ncols + g][tid] = x == 0xFFu ? INT64_MIN : (int64_t)x;
+                m &= s_tab[ld.fgtab[j]][x];
+            }
+            if (!((m >> LT_COMMON) & 1u) || (a.pred.nconj > 0 && !(m & ((1u << a.pred.nconj) - 1)))) return;
+        } else {
+            late_load(a, ld.pref1, row, s_v, tid, pol_s, pol_d);
+        }
+        rest_row(row);
     };
     auto drain = [&](int k) {  // fold the top k (<= 32) queued rows
         __syncwarp();
@@ -4125,6 +4170,32 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
             if (A.a_kind[g] != VD_AGG_COUNT)
                 for (int f = 0; f < A.a_nf[g]; ++f)
                     if (A.a_col[g][f] >= 0) ref(L.aref, A.a_col[g][f]);
+        // fast first round: pref1 = one int32 FK column + u8 lookups through
+        // it whose constraints all became tables
+        L.nfg = 0;
+        L.fk_col = -1;
+        if (ok && A.pred.nconj <= LT_COMMON) {
+            const uint32_t base1 = L.pref1 & ((1u << ncols) - 1), gat1 = L.pref1 >> ncols;
+            bool fast = base1 != 0 && (base1 & (base1 - 1)) == 0 && gat1 != 0;
+            const int fkc = fast ? __builtin_ctz(base1) : -1;
+            fast = fast && cols[fkc].dtype == VD_I32;
+            for (int g = 0; g < A.ngathers && fast; ++g) {
+                if (!((gat1 >> g) & 1u)) continue;
+                int k = -1;
+                for (int h = 0; h < L.ntab; ++h) k = L.tref[h] == ncols + g ? h : k;
+                fast = A.g_fk[g] == fkc && A.g_dt[g] == VD_U8 && k >= 0;
+                if (fast) { L.fg[L.nfg] = g; L.fgtab[L.nfg] = k; ++L.nfg; }
+            }
+            // every constraint on the first-round references is tabulated
+            for (int c = 0; c <= VD_MAX_CONJ && fast; ++c) {
+                if (c >= A.pred.nconj && c != VD_MAX_CONJ) continue;
+                for (int k = 0; k < L.ncons[c] && fast; ++k) fast = !((L.pref1 >> L.cons[c][k].ref) & 1u);
+            }
+            if (fast) L.fk_col = fkc;
+            else L.nfg = 0;
+        }
+        if (const char* fv = getenv("VD_LATE_FAST"))
+            if (strcmp(fv, "0") == 0) L.nfg = 0;
         L.grab = 8;  // measured: 4 and 8 best (0.69 ms at SF100), 64 = static-like (0.76)
         if (const char* gv = getenv("VD_LATE_GRAB")) L.grab = (uint32_t)std::max(1, atoi(gv));
         // the late loads are integer (epsilon = INT64_MIN after widening)
@@ -4142,13 +4213,18 @@ static vd_status try_gf(const vd_pipeline* p, const vd_column* cols, int ncols, 
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }
         // (the attribute is per device context: set on every launch, as for
         // the other dynamic-shared-memory fragments)
-#define LT_GO1(N8_, I32_, CP_)                                                                              \
+#define LT_GO1(N8_, I32_, PV_)                                                                              \
     do {                                                                                                    \
-        e = cudaFuncSetAttribute(k_pipe_late<N8_, I32_, CP_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
+        e = cudaFuncSetAttribute(k_pipe_late<N8_, I32_, PV_>, cudaFuncAttributeMaxDynamicSharedMemorySize, LT_SMEM_MAX); \
         if (e != cudaSuccess) { set_error(cudaGetErrorString(e)); return VD_E_CUDA; }                     \
-        k_pipe_late<N8_, I32_, CP_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);          \
+        k_pipe_late<N8_, I32_, PV_><<<grid, LT_THREADS, lsm, s>>>(A, L, parts, dn, (Slot16*)out);          \
     } while (0)
-#define LT_GO(N8_, I32_) do { if (L.ncons[0] >= 0) LT_GO1(N8_, I32_, true); else LT_GO1(N8_, I32_, false); } while (0)
+#define LT_GO(N8_, I32_)                                                                                    \
+    do {                                                                                                    \
+        if (L.ncons[0] < 0) LT_GO1(N8_, I32_, 0);                                                           \
+        else if (L.nfg > 0) LT_GO1(N8_, I32_, 2);                                                           \
+        else LT_GO1(N8_, I32_, 1);                                                                          \
+    } while (0)
         if (n8 == 2) { if (i32) LT_GO(2, true); else LT_GO(2, false); }
         else if (n8 == 1) { if (i32) LT_GO(1, true); else LT_GO(1, false); }
         else LT_GO(0, true);

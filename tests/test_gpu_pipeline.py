@@ -175,6 +175,9 @@ def test_fkj_q19_vs_oracle(sel_mode, generic, n):
     got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews, want=frag)[0], plan)
     assert {k: tuple(v[:2]) for k, v in got.items()} == exp
     if sel_mode == vd.VD_SEL_BRANCH and not generic:
+        with env(VD_LATE_FAST="0"):  # the late fragment without its fast first round
+            got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews, want=("late",))[0], plan)
+        assert {k: tuple(v[:2]) for k, v in got.items()} == exp
         with env(VD_LATE="off"):  # the dense star-join fragment on the same plan
             got = vd.decode_partials(run(plan, views, len(li["l_partkey"]), dviews, want=("star_join",))[0], plan)
         assert {k: tuple(v[:2]) for k, v in got.items()} == exp
@@ -670,9 +673,10 @@ def test_late_fragment_selectivity_estimate():
                 assert vd.decode_partials(got, plan) == exp
 
 
+@pytest.mark.parametrize("late_fast", ["1", "0"])
 @pytest.mark.parametrize("n", [1, 15, 16, 17, 511, 513, 4099])
 @pytest.mark.parametrize("lead", ["none", "all", "some"])
-def test_late_fragment_edge_sizes(n, lead):
+def test_late_fragment_edge_sizes(n, lead, late_fast):
     """Late fragment at sizes around its 16-row lead words and 32-row drains
     (tail rows only, one word, one word + tail, partial drains) with leads
     that pass nothing, everything or some rows; against the interpreter
@@ -707,13 +711,14 @@ cnt := FoldCount(positions)
     exp = {0: [p.get("total")[0], c, c]} if c else {}
     keep, views = load([a, fk, x])
     dkeep, dviews = load([d])
-    with env(VD_LATE="force"):
+    with env(VD_LATE="force", VD_LATE_FAST=late_fast):
         got, _ = run(plan, views, n, dviews, want=("late",))
     assert vd.decode_partials(got, plan) == exp
 
 
+@pytest.mark.parametrize("late_fast", ["1", "0"])
 @pytest.mark.parametrize("seed", range(12))
-def test_late_fragment_random_fk_plans_vs_oracle(seed):
+def test_late_fragment_random_fk_plans_vs_oracle(seed, late_fast):
     """Late fragment with FK lookups on random branching plans: a common u8
     lead on the fact table, per-conjunction terms on two u8 dimension columns
     (acceptance tables: every comparison kind, IN sets, NE, codes >= 64), an
@@ -780,7 +785,7 @@ def test_late_fragment_random_fk_plans_vs_oracle(seed):
     dkeep, dviews = load([d1, d2, dr])
     plan = vd.pipeline(pred_=vd.pred([[(ref_idx[k], cmp, val) for k, cmp, val in t] for t in conjs]),
                        gathers=[(0, 0, 1), (0, 1, 1), (0, 2, 1)], aggs=[("sum", [3]), ("count",)])
-    with env(VD_LATE="force"):
+    with env(VD_LATE="force", VD_LATE_FAST=late_fast):  # the fast first round (FK + tabulated u8 lookups) or not
         got = vd.decode_partials(run(plan, views, n, dviews, want=("late",))[0], plan)
     assert got == exp
     with env(VD_LATE="off", VD_STAR_VARIANT="off"):  # the dense gather-fold fragment agrees
