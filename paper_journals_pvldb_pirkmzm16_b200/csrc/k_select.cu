@@ -1148,11 +1148,14 @@ constexpr int SL_STG = 512 + 128 + 60;        // per-warp position stage (ints):
                                               // VD_SEL_MID lane-owned positions + pad; the last 32: the words
 static_assert(3 + 512 + 128 + 4 <= SL_STG - 32, "dense stage");
 constexpr int SL_SPARSE = 48;                 // defaults: branching chunks this sparse store directly,
-constexpr int SL_MID = 320;                   // ... this sparse: lane-owned rows, staged;
+constexpr int SL_UNROLL = 160;                // ... this sparse: lane-owned rows, a per-bit loop (staged),
+constexpr int SL_MID = 640;                   // ... this sparse: lane-owned rows, a fixed 32-row loop with
+                                              //     predicated stores (staged); denser: ballot blocks
 constexpr int SL_MID_PRED = 640;              // predicated chunks this sparse: lane-owned cursor arithmetic
-                                              // (VD_SEL_SPARSE / VD_SEL_MID override; measured at s = 0.5:
-                                              // predicated 0.89 ms lane-owned vs 1.05 ms ballot blocks,
-                                              // branching 0.97 either way)
+                                              // (VD_SEL_SPARSE / VD_SEL_UNROLL / VD_SEL_MID override;
+                                              // measured at s = 0.5: predicated 0.89 ms lane-owned vs 1.05 ms
+                                              // ballot blocks; branching 0.87 ms with the fixed loop vs 0.97
+                                              // per-bit loop or ballot blocks, profiles/round2s3_fig1_selpos_lag.md)
 static_assert(640 + 4 + (640 + 4) / 32 + 4 <= SL_STG - 32, "lane-owned stage (VD_SEL_MID <= 640)");
 
 struct SlShared {
@@ -1212,7 +1215,8 @@ __device__ __forceinline__ void sl_flush(const int32_t* sw, int a, int tot, int3
 // row0 + 32 L + i), `cnt` its population, o = the chunk's first output.
 template <int MODE>
 __device__ __forceinline__ void sl_decode(uint32_t word, int cnt, int32_t* __restrict__ o, int32_t row0,
-                                          int32_t* __restrict__ sw, int lane, int sparse_max, int mid_max) {
+                                          int32_t* __restrict__ sw, int lane, int sparse_max, int mid_max,
+                                          int unroll_min) {
     const unsigned lt = lanemask_lt();
     if (MODE == 1 && cnt <= mid_max) {
         // predicated, lane-owned rows: cursor arithmetic over the lane's 32
@@ -1260,6 +1264,24 @@ __device__ __forceinline__ void sl_decode(uint32_t word, int cnt, int32_t* __res
                 ++k;
                 m &= m - 1;
             }
+            return;
+        }
+        if (cnt > unroll_min) {
+            // denser lane-owned chunks: the lane walks all 32 rows with the
+            // store under the row's predicate (only qualifying rows are
+            // written: branching) -- a fixed loop, no divergence on the
+            // per-lane bit counts; then 16-byte stores
+            const int a = (int)(((uintptr_t)o >> 2) & 3);
+            int cur = k + a;
+#pragma unroll
+            for (int i = 0; i < 32; ++i) {
+                const uint32_t f = (word >> i) & 1u;
+                if (f) sw[cur] = r + 1 + i;
+                cur += f;
+            }
+            __syncwarp();
+            sl_flush(sw, a, cnt, o, lane);
+            __syncwarp();
             return;
         }
         // lane-owned rows staged (index x at x + x/32: lanes 32 apart hit
@@ -1333,7 +1355,7 @@ template <int MODE, typename T, int LAG>
 __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__ col, T lo, T hi, int64_t n,
                                                            int32_t* __restrict__ out, int64_t* __restrict__ out_count,
                                                            unsigned int* __restrict__ cnt /* [nk][G], zeroed */,
-                                                           int sparse_max, int mid_max) {
+                                                           int sparse_max, int mid_max, int unroll_min) {
     static_assert(sizeof(T) == 4, "k_sel_lag: 4-byte columns (f32 / i32)");
     static_assert(SL_PUB < SL_BASE && SL_BASE < LAG && LAG + SL_STAGES + 1 <= SL_NS, "k_sel_lag: lags / shared slots");
     constexpr uint32_t TB = SL_CW * 1024 * sizeof(T);
@@ -1503,7 +1525,7 @@ __global__ void __launch_bounds__(SL_THREADS, 1) k_sel_lag(const T* __restrict__
             if (cd > 0) {
                 const int64_t ob = H.base[ds] + H.off[ds][warp];
                 const int32_t row0 = (int32_t)(((kd * G + c) * SL_CW + warp) * 1024);
-                sl_decode<MODE>(q[0], cd, out + ob, row0, sw, lane, sparse_max, mid_max);
+                sl_decode<MODE>(q[0], cd, out + ob, row0, sw, lane, sparse_max, mid_max, unroll_min);
             }
         }
     }
@@ -1551,8 +1573,9 @@ static cudaError_t run_select_lag(const T* col, T lo, T hi, int64_t n, int32_t* 
     };
     // lane-owned chunks must fit the stage: x + x/32 + 4 < SL_STG
     int sparse_max = knob("VD_SEL_SPARSE", SL_SPARSE, 1024), mid_max = knob("VD_SEL_MID", MODE ? SL_MID_PRED : SL_MID, 640);
-    void* args[] = {(void*)&col,       (void*)&lo,  (void*)&hi,         (void*)&n,      (void*)&out_pos,
-                    (void*)&out_count, (void*)&cnt, (void*)&sparse_max, (void*)&mid_max};
+    int unroll_min = knob("VD_SEL_UNROLL", SL_UNROLL, 1024);  // branching lane-owned chunks above this: the fixed loop
+    void* args[] = {(void*)&col,       (void*)&lo,  (void*)&hi,         (void*)&n,       (void*)&out_pos,
+                    (void*)&out_count, (void*)&cnt, (void*)&sparse_max, (void*)&mid_max, (void*)&unroll_min};
     e = cudaLaunchCooperativeKernel((const void*)kern, dim3(G), dim3(SL_THREADS), args, sm, s);
     ++*nl;
     return e;

@@ -117,13 +117,14 @@ def test_large_select_kernels_vs_oracle(mode, n, t):
 
 
 @pytest.mark.parametrize("mode", ["branch", "predicated"])
-@pytest.mark.parametrize("mid", [None, "0", "640"])
+@pytest.mark.parametrize("mid", [None, "0", "640/1024", "640/100"])
 def test_lag_select_chunk_density_mix(mode, mid):
     """Chunks of every density class of k_sel_lag's decode in one input
     (empty, <= SL_SPARSE, lane-owned, dense ballot blocks, full) with NaN
-    epsilon rows, i32 and f32, against the oracle; the lane-owned threshold
-    at its default, off (every chunk through the ballot blocks) and at its
-    maximum."""
+    epsilon rows, i32 and f32, against the oracle; the thresholds at their
+    defaults, lane-owned off (every chunk through the ballot blocks), and
+    lane-owned up to its maximum with the per-bit loop only / the fixed
+    32-row loop above 100 positions."""
     n = 148 * 15 * 1024 * 6 + 12345
     rng = np.random.default_rng(7)
     chunk = np.arange(n) // 1024
@@ -132,7 +133,10 @@ def test_lag_select_chunk_density_mix(mode, mid):
     v[::977] = np.nan
     pos_o, cnt_o, _ = oracle.select_f32(v, 0.5, "lt")
     fn = vd.select_branch if mode == "branch" else vd.select_predicated
-    with env(**({} if mid is None else {"VD_SEL_MID": mid})):
+    knobs = {} if mid is None else {"VD_SEL_MID": mid.split("/")[0]}
+    if mid and "/" in mid:  # branching chunks above 100 positions through the fixed lane loop
+        knobs["VD_SEL_UNROLL"] = mid.split("/")[1]
+    with env(**knobs):
         _density_mix_check(fn, v, n, pos_o, cnt_o)
 
 
